@@ -1,0 +1,336 @@
+#!/usr/bin/env python
+"""Benchmark of the rigid-docking hot path (BASELINE.json metric: probe rotations scored/sec
+at a 128^3 grid, plus % of the FP32 roofline).
+
+Workload (BASELINE configs[2], "FTMap production"): 128^3 receptor at 0.8 A, P = 4 terms,
+16 probes x 500 rotations (m = 4), top-4 poses per rotation, exclusion radius rho = 1.
+One step = one dock_probe_batch over this rank's share of the 8000 (probe, rotation) units
+(voxelize + correlate + weighted score + per-rotation filter) and, for N > 1, the single
+NCCL all-gather of the pose blocks.  Inputs are synthetic (dockgen, seeded).
+
+    python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference]
+
+Prints ONE JSON line on rank 0.  ``--impl reference`` times the FP64 CPU oracle (the
+reference arm of this tier) on bounded samples of the same workload.
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import statistics
+import subprocess
+import sys
+import threading
+import time
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+import numpy as np  # noqa: E402
+
+import dockgen as g  # noqa: E402
+
+METRIC = "probe rotations scored/sec at 128^3 grid (1/2/4/8 B200); % FP32 peak"
+UNIT = "probe rotations/s"
+
+
+def parse():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=5)
+    ap.add_argument("--warmup", type=int, default=3)
+    ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
+    ap.add_argument("--config", default="prod", choices=sorted(g.CONFIGS))
+    ap.add_argument("--k", type=int, default=None)
+    ap.add_argument("--rho", type=int, default=1)
+    ap.add_argument("--no-e2e", action="store_true")
+    ap.add_argument("--no-cpu-baseline", action="store_true")
+    ap.add_argument("--cpu-seconds", type=float, default=12.0, help="target oracle sample duration")
+    ap.add_argument("--regions", type=int, default=0)
+    return ap.parse_args()
+
+
+def workload(cfg_name: str, k_override, rho: int):
+    c = g.CONFIGS[cfg_name]
+    k = k_override or c.k
+    R = g.receptor_ftmap_like(c.n, c.P)
+    w = g.weights(c.P)
+    probes = g.probes(c.n_probes, c.m, c.P)
+    rot = g.rotations(c.n_rot)
+    desc = {
+        "workload": f"{c.name}: {c.n[0]}x{c.n[1]}x{c.n[2]} receptor at {g.SPACING} A, P={c.P} terms, "
+                    f"{c.n_probes} probes x {c.n_rot} rotations, m={c.m}, top-{k}/rotation, rho={rho}",
+        "grid": list(c.n), "probe_m": c.m, "terms": c.P, "probes": c.n_probes, "rotations": c.n_rot,
+        "units": c.n_probes * c.n_rot, "k": k, "rho": rho, "receptor": "ftmap-like synthetic (seed 1001)",
+    }
+    return c, k, R, w, probes, rot, desc
+
+
+def cpu_cores() -> int:
+    try:
+        return len(os.sched_getaffinity(0))
+    except AttributeError:  # pragma: no cover
+        return os.cpu_count() or 1
+
+
+def oracle_sample(R, w, probes, rot, k, rho, n_units, target_s):
+    """Time the FP64 oracle (as it stands) on a bounded, spread sample of units: blocks of
+    ``cores`` consecutive units (one per OpenMP thread) at evenly spread offsets."""
+    import oracle
+    oracle.build_oracle()
+    cores = cpu_cores()
+    t0 = time.perf_counter()
+    oracle.dock(R, w, g.SPACING, probes, rot, k, rho, unit_begin=0, unit_end=1, n_threads=1)
+    t_unit = max(time.perf_counter() - t0, 1e-3)
+    blocks = int(max(1, min(n_units // cores, round(target_s / t_unit))))
+    offsets = np.linspace(0, n_units - cores, blocks).astype(np.int64)
+    done = 0
+    t0 = time.perf_counter()
+    for b in offsets:
+        e = min(n_units, int(b) + cores)
+        oracle.dock(R, w, g.SPACING, probes, rot, k, rho, unit_begin=int(b), unit_end=e, n_threads=cores)
+        done += e - int(b)
+    dt = time.perf_counter() - t0
+    return {"value": done / dt, "unit": UNIT, "cores": cores, "kind": "oracle",
+            "sample": f"{done} units = {blocks} blocks of {cores} consecutive (probe, rotation) units spread "
+                      f"over the workload; FP64 C oracle (gcc -O2, OpenMP {cores} threads); {dt:.1f} s"}
+
+
+class ClockSampler:
+    """nvidia-smi clocks + throttle reasons sampled every 200 ms during the timed region."""
+    FIELDS = ("clocks.sm,clocks.max.sm,clocks_event_reasons.hw_slowdown,"
+              "clocks_event_reasons.hw_thermal_slowdown,clocks_event_reasons.sw_thermal_slowdown,"
+              "clocks_event_reasons.sw_power_cap")
+
+    def __init__(self, index: int):
+        self.index = index
+        self.proc = None
+        self.lines = []
+
+    def start(self):
+        try:
+            self.proc = subprocess.Popen(
+                ["nvidia-smi", f"--query-gpu={self.FIELDS}", "--format=csv,noheader,nounits", "-i",
+                 str(self.index), "-lms", "200"], stdout=subprocess.PIPE, stderr=subprocess.DEVNULL, text=True)
+            self.t = threading.Thread(target=self._read, daemon=True)
+            self.t.start()
+        except (OSError, FileNotFoundError):
+            self.proc = None
+
+    def _read(self):
+        for line in self.proc.stdout:
+            self.lines.append(line.strip())
+
+    def stop(self):
+        if not self.proc:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["nvidia-smi unavailable"]}
+        time.sleep(0.25)
+        self.proc.terminate()
+        try:
+            self.proc.wait(timeout=2)
+        except subprocess.TimeoutExpired:
+            self.proc.kill()
+        sm, mx, reasons = [], [], set()
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        for line in self.lines:
+            parts = [p.strip() for p in line.split(",")]
+            if len(parts) < 6:
+                continue
+            try:
+                sm.append(float(parts[0]))
+                mx.append(float(parts[1]))
+            except ValueError:
+                continue
+            for nm, v in zip(names, parts[2:6]):
+                if v.lower().startswith("active"):
+                    reasons.add(nm)
+        return {"sm_mhz": statistics.median(sm) if sm else None, "sm_max_mhz": max(mx) if mx else None,
+                "reasons": sorted(reasons), "samples": len(sm)}
+
+
+def run_reference(args):
+    rank = int(os.environ.get("RANK", "0"))
+    if rank != 0:
+        return
+    c, k, R, w, probes, rot, desc = workload(args.config, args.k, args.rho)
+    n_units = c.n_probes * c.n_rot
+    per_step = max(2.0, min(args.cpu_seconds, 120.0 / max(1, args.steps + args.warmup)))
+    samples = []
+    for i in range(args.warmup + args.steps):
+        cb = oracle_sample(R, w, probes, rot, k, args.rho, n_units, per_step)
+        if i >= args.warmup:
+            samples.append(cb)
+    v = statistics.median(s["value"] for s in samples)
+    cb = dict(samples[-1])
+    cb["value"] = v
+    line = {"impl": "reference", "metric": METRIC, "value": v, "unit": UNIT, "n_gpus": args.gpus,
+            "steps": args.steps, "warmup": args.warmup, "ms_per_step": 1000.0 * n_units / v,
+            "higher_is_better": True, "scaling": "strong", "vs_baseline": None, "dtype": "f64",
+            "data": "synthetic", "config": desc, "cpu_baseline": cb,
+            "e2e": {"value": v, "unit": UNIT, "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}
+    print(json.dumps(line), flush=True)
+
+
+def peaks():
+    p = os.path.join(ROOT, "MEASURED_PEAKS.json")
+    if os.path.exists(p):
+        with open(p) as f:
+            return json.load(f), "measured"
+    return {"sm_max_mhz": 1965.0}, "fallback"
+
+
+def run_ours(args):
+    import torch
+    import torch.distributed as dist
+
+    import paper_conf_ipps_sukhwanih10_b200 as D
+    from paper_conf_ipps_sukhwanih10_b200 import parallel
+
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    torch.cuda.set_device(local)
+    if world > 1:
+        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+    dev = torch.device("cuda", local)
+
+    c, k, R, w, probes, rot, desc = workload(args.config, args.k, args.rho)
+    n_units = c.n_probes * c.n_rot
+    b, e = parallel.shard_range(n_units, rank, world)
+    ctx = D.dock_init(torch.from_numpy(R).to(dev), torch.from_numpy(w).to(dev), g.SPACING, m_max=c.m,
+                      device=local)
+    if args.regions:
+        D.dock_set_tuning(ctx, D.DOCK_TUNE_REGIONS, args.regions)
+    probes_dev = [{"xyz": torch.from_numpy(p.xyz).to(dev), "coef": torch.from_numpy(p.coef).to(dev), "m": p.m}
+                  for p in probes]
+    rot_dev = torch.from_numpy(rot).to(dev)
+    out = torch.empty((e - b, k, 4), dtype=torch.int32, device=dev)
+    l2 = int(D.dock_get_info(ctx)["l2_bytes"]) or (126 << 20)
+    flush = torch.empty(max(2 * l2, 256 << 20) // 4, dtype=torch.float32, device=dev)
+    stream = torch.cuda.current_stream(dev)
+
+    def step():
+        D.dock_probe_batch(ctx, probes_dev, rot_dev, b, e, k, args.rho, out=out)
+        if world > 1:
+            parallel.gather_poses(out, n_units)
+
+    for _ in range(args.warmup):
+        step()
+    torch.cuda.synchronize()
+    if world > 1:
+        dist.barrier()
+    torch.cuda.synchronize()
+    clk = ClockSampler(local)
+    clk.start()
+    times, corr, launches, fallbacks = [], [], 0, 0
+    for i in range(args.steps):
+        flush.fill_(float(i))            # L2 flush between timed steps (outside the events)
+        e0 = torch.cuda.Event(enable_timing=True)
+        e1 = torch.cuda.Event(enable_timing=True)
+        e0.record(stream)
+        step()
+        e1.record(stream)
+        e1.synchronize()
+        times.append(e0.elapsed_time(e1))
+        info = D.dock_get_info(ctx)
+        corr.append(info["corr_ms_last"])
+        launches += int(info["kernels_last"])
+        fallbacks += int(info["fallback_last"])
+    torch.cuda.synchronize()
+    if world > 1:
+        dist.barrier()
+    torch.cuda.synchronize()
+    clocks = clk.stop()
+    t_local = sum(times)
+    t = torch.tensor([t_local, sum(corr)], dtype=torch.float64, device=dev)
+    if world > 1:
+        dist.all_reduce(t, op=dist.ReduceOp.MAX)
+    t_max, corr_max = float(t[0]), float(t[1])
+    ms_step = t_max / args.steps
+    value = n_units / (ms_step / 1000.0)
+
+    # ---- e2e through the public API with host buffers (H2D of inputs + D2H of poses inside)
+    e2e = None
+    if not args.no_e2e:
+        h2d = rot.nbytes + sum(p.xyz.nbytes + p.coef.nbytes for p in probes) + 4 * (len(probes) + 1)
+        d2h = n_units * k * 16
+        out2 = torch.empty((e - b, k, 4), dtype=torch.int32, device=dev)
+
+        def step_e2e():
+            D.dock_probe_batch(ctx, probes, rot, b, e, k, args.rho, out=out2)
+            full = parallel.gather_poses(out2, n_units) if world > 1 else out2
+            if rank == 0:
+                full.cpu()
+
+        step_e2e()
+        torch.cuda.synchronize()
+        et = []
+        for i in range(args.steps):
+            flush.fill_(float(i))
+            torch.cuda.synchronize()
+            t0 = time.perf_counter()
+            step_e2e()
+            torch.cuda.synchronize()
+            et.append(time.perf_counter() - t0)
+        tt = torch.tensor([sum(et)], dtype=torch.float64, device=dev)
+        if world > 1:
+            dist.all_reduce(tt, op=dist.ReduceOp.MAX)
+        e2e = {"value": n_units / (float(tt[0]) / args.steps), "unit": UNIT, "h2d_bytes_per_step": int(h2d),
+               "d2h_bytes_per_step": int(d2h), "timer": "host wall clock around the synchronous API call"}
+
+    # ---- roofline of the dominant kernel (k_corr): plain FP32 FFMA pipe (bound "alu")
+    pk, pk_kind = peaks()
+    sm_max = float(pk.get("sm_max_mhz", 1965.0))
+    info = D.dock_get_info(ctx)
+    n_sms = int(info["n_sms"])
+    peak_tflops = n_sms * 128 * 2 * sm_max * 1e6 / 1e12
+    units_local = e - b
+    flops_launch = 2.0 * c.P * c.m ** 3 * c.n[0] * c.n[1] * c.n[2] * units_local
+    corr_ms = corr_max / args.steps
+    achieved = flops_launch / (corr_ms / 1000.0) / 1e12
+    traffic = None
+    tp = os.path.join(ROOT, "profiles", "corr_traffic.json")
+    if os.path.exists(tp):
+        with open(tp) as f:
+            tj = json.load(f)
+        if tj.get("config") == args.config and tj.get("gpus") == world:
+            traffic = tj.get("dram_bytes_per_launch")
+    roof = {"bound": "alu", "kernel": "k_corr<4,false>", "achieved": achieved, "peak": peak_tflops,
+            "unit": "TFLOP/s", "frac": achieved / peak_tflops, "traffic": traffic,
+            "peak_source": f"{n_sms} SMs x 128 FP32 lanes x 2 FLOP x {sm_max:.0f} MHz "
+                           f"(sm_max_mhz from MEASURED_PEAKS.json: {pk_kind})",
+            "flops_per_launch": flops_launch, "launch_ms": corr_ms,
+            "kernel_share_of_step": corr_ms / ms_step if ms_step > 0 else None}
+
+    cpu = None
+    if rank == 0 and world == 1 and not args.no_cpu_baseline:
+        cpu = oracle_sample(R, w, probes, rot, k, args.rho, n_units, args.cpu_seconds)
+
+    if rank == 0:
+        desc = dict(desc)
+        desc.update({"parallelism": f"rotation-shard x{world}" if world > 1 else "single GPU",
+                     "l2": f"flushed between timed steps ({flush.numel() * 4 >> 20} MiB write); "
+                           f"receptor {R.nbytes >> 20} MiB fits in L2",
+                     "regions": info["regions_last"], "items": info["items_last"],
+                     "fallback_rotations": fallbacks, "timing": "CUDA events on the context stream"})
+        line = {"metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world, "steps": args.steps,
+                "warmup": args.warmup, "ms_per_step": ms_step, "higher_is_better": True, "scaling": "strong",
+                "vs_baseline": None, "dtype": "f32", "data": "synthetic", "config": desc,
+                "e2e": e2e, "gpu_launches": launches, "roofline": roof, "cpu_baseline": cpu, "clocks": clocks}
+        print(json.dumps(line), flush=True)
+    D.dock_destroy(ctx)
+    if world > 1:
+        dist.destroy_process_group()
+
+
+def main():
+    args = parse()
+    if args.impl == "reference":
+        run_reference(args)
+    else:
+        run_ours(args)
+
+
+if __name__ == "__main__":
+    main()

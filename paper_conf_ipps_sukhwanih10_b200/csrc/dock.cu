@@ -1,0 +1,891 @@
+// dock.cu -- host implementation of the C ABI in include/dock.h (libdock.so).
+//
+// Owns the device memory layout (cyclic-halo padded receptor, TMA descriptors,
+// per-call scratch), validates arguments, plans launches and runs
+//   reset -> k_voxelize -> k_corr<M, top-k> -> k_merge [-> exact fallback]
+// on the context's stream.  Citations "P:L.." point into PAPER.md.
+#include <cuda.h>
+#include <cuda_runtime.h>
+#include <cudaTypedefs.h>
+
+#include <algorithm>
+#include <cmath>
+#include <cstdarg>
+#include <cstdio>
+#include <cstring>
+#include <new>
+#include <vector>
+
+#include "dock.h"
+#include "dock_kernels.cuh"
+
+static_assert(sizeof(dock_pose) == 16, "dock_pose must be 16 bytes");
+static_assert(sizeof(dk::PoseOut) == sizeof(dock_pose), "kernel pose layout mismatch");
+
+namespace {
+
+constexpr int kSmemLimit = 227 * 1024;
+
+struct DevBuf {
+    void* p = nullptr;
+    size_t cap = 0;
+};
+
+struct MPlan {                 // per-probe-size launch plan
+    bool ok = false;
+    CUtensorMap tmap;
+    int TXB = 0, TYB = 0, TZB = 0;
+    int stage_rec_bytes = 0, stage_bytes = 0, nstage = 0, smem = 0;
+};
+
+}  // namespace
+
+struct dock_ctx {
+    int device = 0;
+    cudaStream_t stream = nullptr;
+    bool own_stream = false;
+    int nx = 0, ny = 0, nz = 0, P = 0, m_max = 0;
+    float spacing = 0.f;
+    int n_sms = 148;
+    double l2_bytes = 0;
+    dk::Geo geo{};
+    float* d_rec = nullptr;
+    float* d_w = nullptr;      // [P] weights
+    float* d_eye = nullptr;    // [P][P] identity (per-term grids)
+    float* d_ones = nullptr;   // [P] ones (unweighted voxel export)
+    MPlan plan[DOCK_MAX_M + 1];
+    // per-call scratch (grow-only)
+    DevBuf xyz, coef, off, rot, Lw, T, mu, cnt, cand, poses, fb_list, grid, slots, units, Lw_fb;
+    int* d_small = nullptr;    // [0] status, [1] fb_cnt, [2] cand_max
+    int* h_small = nullptr;    // pinned mirror
+    void* h_stage = nullptr;   // pinned staging for host inputs
+    size_t h_stage_cap = 0;
+    // tuning
+    int regions_override = 0;
+    int force_fallback = 0;
+    int cand_cap = 1024;
+    // stats
+    int regions_last = 0;
+    int64_t items_last = 0, fallback_last = 0, cand_max_last = 0, kernels_last = 0;
+    cudaEvent_t ev_corr[2] = {nullptr, nullptr};   // bracket the k_corr launch of dock_probe_batch
+    bool ev_corr_valid = false;
+    bool dead = false;
+    char err[512] = {0};
+};
+
+namespace {
+
+dock_status fail(dock_ctx* c, dock_status s, const char* fmt, ...)
+{
+    if (c) {
+        va_list ap;
+        va_start(ap, fmt);
+        vsnprintf(c->err, sizeof(c->err), fmt, ap);
+        va_end(ap);
+        if (s == DOCK_E_CUDA) c->dead = true;
+    }
+    return s;
+}
+
+#define CU(call)                                                                                        \
+    do {                                                                                                \
+        cudaError_t e_ = (call);                                                                        \
+        if (e_ != cudaSuccess) {                                                                        \
+            return fail(ctx, e_ == cudaErrorMemoryAllocation ? DOCK_E_OOM : DOCK_E_CUDA, "%s: %s (%s:%d)", \
+                        #call, cudaGetErrorString(e_), __FILE__, __LINE__);                             \
+        }                                                                                               \
+    } while (0)
+
+#define TRY(expr)                          \
+    do {                                   \
+        dock_status s_ = (expr);           \
+        if (s_ != DOCK_OK) return s_;      \
+    } while (0)
+
+bool is_device_ptr(const void* p)
+{
+    if (!p) return false;
+    cudaPointerAttributes at;
+    if (cudaPointerGetAttributes(&at, p) != cudaSuccess) {
+        cudaGetLastError();
+        return false;
+    }
+    return at.type == cudaMemoryTypeDevice || at.type == cudaMemoryTypeManaged;
+}
+
+dock_status ensure(dock_ctx* ctx, DevBuf& b, size_t bytes)
+{
+    if (bytes <= b.cap) return DOCK_OK;
+    if (b.p) CU(cudaFree(b.p));
+    b.p = nullptr;
+    b.cap = 0;
+    size_t want = std::max<size_t>(bytes, 256);
+    CU(cudaMalloc(&b.p, want));
+    b.cap = want;
+    return DOCK_OK;
+}
+
+dock_status ensure_pinned(dock_ctx* ctx, size_t bytes)
+{
+    if (bytes <= ctx->h_stage_cap) return DOCK_OK;
+    if (ctx->h_stage) {
+        CU(cudaStreamSynchronize(ctx->stream));
+        CU(cudaFreeHost(ctx->h_stage));
+    }
+    ctx->h_stage = nullptr;
+    ctx->h_stage_cap = 0;
+    size_t want = std::max<size_t>(bytes, 1 << 16);
+    CU(cudaHostAlloc(&ctx->h_stage, want, cudaHostAllocDefault));
+    ctx->h_stage_cap = want;
+    return DOCK_OK;
+}
+
+int round_up(int v, int a) { return (v + a - 1) / a * a; }
+
+PFN_cuTensorMapEncodeTiled_v12000 encode_fn()
+{
+    static PFN_cuTensorMapEncodeTiled_v12000 fn = nullptr;
+    if (!fn) {
+        void* p = nullptr;
+        cudaDriverEntryPointQueryResult q;
+        if (cudaGetDriverEntryPoint("cuTensorMapEncodeTiled", &p, cudaEnableDefault, &q) == cudaSuccess &&
+            q == cudaDriverEntryPointSuccess)
+            fn = reinterpret_cast<PFN_cuTensorMapEncodeTiled_v12000>(p);
+        else
+            cudaGetLastError();
+    }
+    return fn;
+}
+
+// Tile geometry: XT = 8 translations per lane along x, LX lanes per row.  LX is chosen to
+// waste the fewest x translations (ties: wider rows, less halo).
+dk::Geo choose_geo(int nx, int ny, int nz, int m_max)
+{
+    dk::Geo g{};
+    g.nx = nx;
+    g.ny = ny;
+    g.nz = nz;
+    int best = 16;
+    double best_w = 1e30;
+    for (int lx : {16, 8, 4}) {
+        int tx = lx * dk::XT;
+        int ntx = (nx + tx - 1) / tx;
+        double w = double(ntx) * tx / nx;
+        if (w < best_w - 1e-9) {
+            best_w = w;
+            best = lx;
+        }
+    }
+    g.LX = best;
+    g.WY = 32 / best;
+    g.TX = best * dk::XT;
+    int rows = dk::NWC * g.WY;   // 16, 32 or 64
+    g.TY = rows == 16 ? 4 : 8;
+    g.TZ = rows / g.TY;
+    g.ntx = (nx + g.TX - 1) / g.TX;
+    g.nty = (ny + g.TY - 1) / g.TY;
+    g.ntz = (nz + g.TZ - 1) / g.TZ;
+    g.ntiles = g.ntx * g.nty * g.ntz;
+    int txb_max = round_up(g.TX + m_max - 1, 4);
+    g.Xp = round_up((g.ntx - 1) * g.TX + txb_max, 4);
+    g.Yp = g.nty * g.TY + m_max - 1;
+    g.Zp = g.ntz * g.TZ + m_max - 1;
+    return g;
+}
+
+dock_status make_plan(dock_ctx* ctx, int m)
+{
+    MPlan& pl = ctx->plan[m];
+    if (pl.ok) return DOCK_OK;
+    const dk::Geo& g = ctx->geo;
+    pl.TXB = round_up(g.TX + m - 1, 4);
+    pl.TYB = g.TY + m - 1;
+    pl.TZB = g.TZ + m - 1;
+    if (pl.TXB > 256 || pl.TYB > 256 || pl.TZB > 256)
+        return fail(ctx, DOCK_E_UNSUPPORTED, "TMA box too large");
+    pl.stage_rec_bytes = round_up(pl.TXB * pl.TYB * pl.TZB * 4, 128);
+    pl.stage_bytes = round_up(pl.stage_rec_bytes + m * m * m * dk::RB * 4, 128);
+    int ns = (kSmemLimit - 256) / pl.stage_bytes;
+    ns = std::min(ns, 4);
+    if (ns < 2) return fail(ctx, DOCK_E_UNSUPPORTED, "probe grid m=%d too large for the shared-memory ring", m);
+    pl.nstage = ns;
+    pl.smem = ns * pl.stage_bytes + 2 * ns * 8;
+    auto fn = encode_fn();
+    if (!fn) return fail(ctx, DOCK_E_CUDA, "cuTensorMapEncodeTiled unavailable");
+    cuuint64_t dims[4] = {(cuuint64_t)g.Xp, (cuuint64_t)g.Yp, (cuuint64_t)g.Zp, (cuuint64_t)ctx->P};
+    cuuint64_t strides[3] = {(cuuint64_t)g.Xp * 4, (cuuint64_t)g.Xp * g.Yp * 4, (cuuint64_t)g.Xp * g.Yp * g.Zp * 4};
+    cuuint32_t box[4] = {(cuuint32_t)pl.TXB, (cuuint32_t)pl.TYB, (cuuint32_t)pl.TZB, 1};
+    cuuint32_t es[4] = {1, 1, 1, 1};
+    CUresult r = fn(&pl.tmap, CU_TENSOR_MAP_DATA_TYPE_FLOAT32, 4, ctx->d_rec, dims, strides, box, es,
+                    CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_L2_256B,
+                    CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+    if (r != CUDA_SUCCESS) return fail(ctx, DOCK_E_CUDA, "cuTensorMapEncodeTiled failed (%d)", (int)r);
+    pl.ok = true;
+    return DOCK_OK;
+}
+
+template <int M, bool GRID>
+cudaError_t launch_corr_t(const MPlan& pl, const dk::CorrArgs& a, int grid, cudaStream_t st)
+{
+    auto kern = dk::k_corr<M, GRID>;
+    cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, pl.smem);
+    if (e != cudaSuccess) return e;
+    kern<<<grid, dk::NTHREADS, pl.smem, st>>>(pl.tmap, a);
+    return cudaGetLastError();
+}
+
+template <bool GRID>
+cudaError_t launch_corr(int m, const MPlan& pl, const dk::CorrArgs& a, int grid, cudaStream_t st)
+{
+    switch (m) {
+        case 1: return launch_corr_t<1, GRID>(pl, a, grid, st);
+        case 2: return launch_corr_t<2, GRID>(pl, a, grid, st);
+        case 3: return launch_corr_t<3, GRID>(pl, a, grid, st);
+        case 4: return launch_corr_t<4, GRID>(pl, a, grid, st);
+        case 5: return launch_corr_t<5, GRID>(pl, a, grid, st);
+        case 6: return launch_corr_t<6, GRID>(pl, a, grid, st);
+        case 7: return launch_corr_t<7, GRID>(pl, a, grid, st);
+        case 8: return launch_corr_t<8, GRID>(pl, a, grid, st);
+        default: return cudaErrorInvalidValue;
+    }
+}
+
+// Regions per rotation batch: minimise waves * (tiles per item + per-item overhead).
+int choose_regions(const dock_ctx* ctx, int64_t n_batches)
+{
+    if (ctx->regions_override > 0) return std::min(ctx->regions_override, ctx->geo.ntiles);
+    const int nt = ctx->geo.ntiles;
+    int best = 1;
+    double best_cost = 1e300;
+    for (int G = 1; G <= std::min(nt, 256); G++) {
+        int tpr = (nt + G - 1) / G;
+        int geff = (nt + tpr - 1) / tpr;
+        int64_t items = n_batches * geff;
+        int64_t waves = (items + ctx->n_sms - 1) / ctx->n_sms;
+        double cost = double(waves) * (tpr + 0.5);
+        if (cost < best_cost - 1e-9) {
+            best_cost = cost;
+            best = geff;
+        }
+    }
+    return best;
+}
+
+dock_status check_ctx(dock_ctx* ctx)
+{
+    if (!ctx) return DOCK_E_INVALID_ARG;
+    if (ctx->dead) return fail(ctx, DOCK_E_CUDA, "context unusable after an earlier CUDA error");
+    cudaError_t e = cudaSetDevice(ctx->device);
+    if (e != cudaSuccess) return fail(ctx, DOCK_E_CUDA, "cudaSetDevice: %s", cudaGetErrorString(e));
+    return DOCK_OK;
+}
+
+// Stage probes (atoms packed probe by probe) and rotations on the device.
+// Returns device pointers in *xyz, *coef, *off, *rot.
+dock_status stage_inputs(dock_ctx* ctx, const dock_probe_desc* probes, int n_probes, const double* rot,
+                         int n_rot, const double** d_xyz, const float** d_coef, const int** d_off,
+                         const double** d_rot)
+{
+    const int P = ctx->P;
+    std::vector<int> off(n_probes + 1, 0);
+    for (int i = 0; i < n_probes; i++) off[i + 1] = off[i] + probes[i].n_atoms;
+    const int na = off[n_probes];
+    const bool rot_dev = is_device_ptr(rot);
+    size_t b_xyz = sizeof(double) * 3 * std::max(na, 1), b_coef = sizeof(float) * P * std::max(na, 1);
+    size_t b_off = sizeof(int) * (n_probes + 1), b_rot = rot_dev ? 0 : sizeof(double) * 9 * n_rot;
+    TRY(ensure(ctx, ctx->xyz, b_xyz));
+    TRY(ensure(ctx, ctx->coef, b_coef));
+    TRY(ensure(ctx, ctx->off, b_off));
+    // pinned staging: [off][rot][xyz][coef] (host probes only)
+    size_t o_rot = round_up((int)b_off, 16), o_xyz = o_rot + round_up((int)b_rot, 16);
+    size_t o_coef = o_xyz + b_xyz;
+    TRY(ensure_pinned(ctx, o_coef + b_coef));
+    // the previous call may still read the staging buffer
+    CU(cudaStreamSynchronize(ctx->stream));
+    char* hs = static_cast<char*>(ctx->h_stage);
+    memcpy(hs, off.data(), b_off);
+    CU(cudaMemcpyAsync(ctx->off.p, hs, b_off, cudaMemcpyHostToDevice, ctx->stream));
+    if (!rot_dev) {
+        TRY(ensure(ctx, ctx->rot, b_rot));
+        memcpy(hs + o_rot, rot, b_rot);
+        CU(cudaMemcpyAsync(ctx->rot.p, hs + o_rot, b_rot, cudaMemcpyHostToDevice, ctx->stream));
+        *d_rot = static_cast<const double*>(ctx->rot.p);
+    } else {
+        *d_rot = rot;
+    }
+    for (int i = 0; i < n_probes; i++) {
+        const dock_probe_desc& pr = probes[i];
+        if (pr.n_atoms == 0) continue;
+        double* dx = static_cast<double*>(ctx->xyz.p) + 3 * (size_t)off[i];
+        float* dc = static_cast<float*>(ctx->coef.p) + (size_t)P * off[i];
+        const size_t bx = sizeof(double) * 3 * pr.n_atoms, bc = sizeof(float) * P * pr.n_atoms;
+        if (is_device_ptr(pr.xyz)) {
+            CU(cudaMemcpyAsync(dx, pr.xyz, bx, cudaMemcpyDeviceToDevice, ctx->stream));
+        } else {
+            char* h = hs + o_xyz + sizeof(double) * 3 * (size_t)off[i];
+            memcpy(h, pr.xyz, bx);
+            CU(cudaMemcpyAsync(dx, h, bx, cudaMemcpyHostToDevice, ctx->stream));
+        }
+        if (is_device_ptr(pr.coef)) {
+            CU(cudaMemcpyAsync(dc, pr.coef, bc, cudaMemcpyDeviceToDevice, ctx->stream));
+        } else {
+            char* h = hs + o_coef + sizeof(float) * P * (size_t)off[i];
+            memcpy(h, pr.coef, bc);
+            CU(cudaMemcpyAsync(dc, h, bc, cudaMemcpyHostToDevice, ctx->stream));
+        }
+    }
+    *d_xyz = static_cast<const double*>(ctx->xyz.p);
+    *d_coef = static_cast<const float*>(ctx->coef.p);
+    *d_off = static_cast<const int*>(ctx->off.p);
+    return DOCK_OK;
+}
+
+dock_status validate_probes(dock_ctx* ctx, const dock_probe_desc* probes, int n_probes, int* m_out)
+{
+    if (!probes || n_probes < 1) return fail(ctx, DOCK_E_INVALID_ARG, "no probes");
+    int m = probes[0].m;
+    for (int i = 0; i < n_probes; i++) {
+        const dock_probe_desc& p = probes[i];
+        if (p.n_atoms < 0) return fail(ctx, DOCK_E_INVALID_ARG, "probe %d: n_atoms < 0", i);
+        if (p.n_atoms > 0 && (!p.xyz || !p.coef)) return fail(ctx, DOCK_E_INVALID_ARG, "probe %d: null atoms", i);
+        if (p.m < 1) return fail(ctx, DOCK_E_INVALID_ARG, "probe %d: m < 1", i);
+        if (p.m > ctx->m_max || p.m > DOCK_MAX_M)
+            return fail(ctx, DOCK_E_UNSUPPORTED, "probe %d: m=%d exceeds m_max=%d", i, p.m, ctx->m_max);
+        if (p.m != m) return fail(ctx, DOCK_E_UNSUPPORTED, "probes of different m in one batch");
+        if (!is_device_ptr(p.xyz) && p.n_atoms > 0) {
+            for (int j = 0; j < 3 * p.n_atoms; j++)
+                if (!std::isfinite(p.xyz[j])) return fail(ctx, DOCK_E_INVALID_ARG, "probe %d: non-finite xyz", i);
+        }
+        if (!is_device_ptr(p.coef) && p.n_atoms > 0) {
+            for (int j = 0; j < ctx->P * p.n_atoms; j++)
+                if (!std::isfinite(p.coef[j])) return fail(ctx, DOCK_E_INVALID_ARG, "probe %d: non-finite coef", i);
+        }
+    }
+    *m_out = m;
+    return DOCK_OK;
+}
+
+dock_status check_status_word(dock_ctx* ctx)
+{
+    int st = ctx->h_small[0];
+    if (st & dk::ST_BAD_ROTATION) return fail(ctx, DOCK_E_BAD_ROTATION, "a rotation is not a proper rotation matrix");
+    if (st & dk::ST_OUTSIDE)
+        return fail(ctx, DOCK_E_PROBE_OUTSIDE_GRID, "a probe atom voxelizes outside the m^3 probe box");
+    return DOCK_OK;
+}
+
+dock_status run_voxelize(dock_ctx* ctx, int m, int n_slots, int64_t unit_begin, const int* d_units, int n_rot,
+                         const double* xyz, const float* coef, const int* off, const double* rot, const float* w,
+                         float* Lw)
+{
+    dk::VoxArgs v{};
+    v.xyz = xyz;
+    v.coef = coef;
+    v.atom_off = off;
+    v.rot = rot;
+    v.w = w;
+    v.unit_list = d_units;
+    v.unit_begin = unit_begin;
+    v.n_rot = n_rot;
+    v.n_slots = n_slots;
+    v.P = ctx->P;
+    v.m = m;
+    v.spacing = ctx->spacing;
+    v.Lw = Lw;
+    v.status = ctx->d_small;
+    int n = n_slots * ctx->P;
+    dk::k_voxelize<<<(n + 127) / 128, 128, 0, ctx->stream>>>(v);
+    CU(cudaGetLastError());
+    ctx->kernels_last++;
+    return DOCK_OK;
+}
+
+dk::CorrArgs corr_args(dock_ctx* ctx, int m, int n_slots, int G, const float* Lw)
+{
+    const MPlan& pl = ctx->plan[m];
+    dk::CorrArgs a{};
+    a.g = ctx->geo;
+    a.P = ctx->P;
+    a.Lw = Lw;
+    a.n_slots = n_slots;
+    a.G = G;
+    a.tiles_per_region = (ctx->geo.ntiles + G - 1) / G;
+    a.nstage = pl.nstage;
+    a.stage_rec_bytes = pl.stage_rec_bytes;
+    a.stage_bytes = pl.stage_bytes;
+    a.TXB = pl.TXB;
+    a.TYB = pl.TYB;
+    a.TZB = pl.TZB;
+    return a;
+}
+
+// Score grids for n slots (GRID epilogue) into grid[n][nz][ny][nx].
+dock_status run_grid(dock_ctx* ctx, int m, int n_slots, const float* Lw, float* grid)
+{
+    int64_t nb = (n_slots + dk::RB - 1) / dk::RB;
+    int G = choose_regions(ctx, nb);
+    dk::CorrArgs a = corr_args(ctx, m, n_slots, G, Lw);
+    a.grid = grid;
+    CU(launch_corr<true>(m, ctx->plan[m], a, (int)(nb * G), ctx->stream));
+    ctx->kernels_last++;
+    return DOCK_OK;
+}
+
+// Exact fallback for flagged slots: full score grid + exact greedy.
+dock_status run_fallback(dock_ctx* ctx, int m, int nfb, int64_t unit_begin, int n_rot, const double* xyz,
+                         const float* coef, const int* off, const double* rot, int k, int rho, void* poses)
+{
+    std::vector<int> slots(nfb);
+    CU(cudaMemcpyAsync(slots.data(), ctx->fb_list.p, sizeof(int) * nfb, cudaMemcpyDeviceToHost, ctx->stream));
+    CU(cudaStreamSynchronize(ctx->stream));
+    std::sort(slots.begin(), slots.end());
+    const size_t ncell = (size_t)ctx->nx * ctx->ny * ctx->nz;
+    const int chunk = (int)std::max<size_t>(1, std::min<size_t>(32, (size_t(1) << 30) / (ncell * 4)));
+    TRY(ensure(ctx, ctx->grid, sizeof(float) * ncell * chunk));
+    TRY(ensure(ctx, ctx->slots, sizeof(int) * 2 * chunk));
+    const int m3 = m * m * m;
+    TRY(ensure(ctx, ctx->Lw_fb, sizeof(float) * ((chunk + dk::RB - 1) / dk::RB) * dk::RB * ctx->P * m3));
+    TRY(ensure_pinned(ctx, sizeof(int) * 2 * chunk));
+    for (int c0 = 0; c0 < nfb; c0 += chunk) {
+        int n = std::min(chunk, nfb - c0);
+        CU(cudaStreamSynchronize(ctx->stream));
+        int* h = static_cast<int*>(ctx->h_stage);
+        for (int i = 0; i < n; i++) {
+            h[i] = (int)(unit_begin + slots[c0 + i]);   // absolute unit
+            h[chunk + i] = slots[c0 + i];                // output slot
+        }
+        CU(cudaMemcpyAsync(ctx->slots.p, h, sizeof(int) * 2 * chunk, cudaMemcpyHostToDevice, ctx->stream));
+        const int* d_units = static_cast<const int*>(ctx->slots.p);
+        const int* d_outslot = d_units + chunk;
+        TRY(run_voxelize(ctx, m, n, 0, d_units, n_rot, xyz, coef, off, rot, ctx->d_w,
+                         static_cast<float*>(ctx->Lw_fb.p)));
+        TRY(run_grid(ctx, m, n, static_cast<const float*>(ctx->Lw_fb.p), static_cast<float*>(ctx->grid.p)));
+        dk::GreedyArgs ga{};
+        ga.grid = static_cast<const float*>(ctx->grid.p);
+        ga.slots = d_outslot;
+        ga.n = n;
+        ga.k = k;
+        ga.rho = rho;
+        ga.n_rot = n_rot;
+        ga.nx = ctx->nx;
+        ga.ny = ctx->ny;
+        ga.nz = ctx->nz;
+        ga.unit_begin = unit_begin;
+        ga.poses = poses;
+        dk::k_greedy_grid<<<n, 1024, 0, ctx->stream>>>(ga);
+        CU(cudaGetLastError());
+        ctx->kernels_last++;
+    }
+    return DOCK_OK;
+}
+
+}  // namespace
+
+// =====================================================================================  ABI
+
+extern "C" {
+
+const char* dock_status_string(dock_status s)
+{
+    switch (s) {
+        case DOCK_OK: return "DOCK_OK";
+        case DOCK_E_INVALID_ARG: return "DOCK_E_INVALID_ARG";
+        case DOCK_E_UNSUPPORTED: return "DOCK_E_UNSUPPORTED";
+        case DOCK_E_PROBE_OUTSIDE_GRID: return "DOCK_E_PROBE_OUTSIDE_GRID";
+        case DOCK_E_BAD_ROTATION: return "DOCK_E_BAD_ROTATION";
+        case DOCK_E_CUDA: return "DOCK_E_CUDA";
+        case DOCK_E_OOM: return "DOCK_E_OOM";
+    }
+    return "DOCK_E_UNKNOWN";
+}
+
+const char* dock_last_error(const dock_ctx* ctx) { return ctx ? ctx->err : "null context"; }
+
+void dock_destroy(dock_ctx* ctx)
+{
+    if (!ctx) return;
+    cudaSetDevice(ctx->device);
+    if (ctx->stream) cudaStreamSynchronize(ctx->stream);
+    DevBuf* bufs[] = {&ctx->xyz, &ctx->coef, &ctx->off, &ctx->rot, &ctx->Lw, &ctx->T, &ctx->mu, &ctx->cnt,
+                      &ctx->cand, &ctx->poses, &ctx->fb_list, &ctx->grid, &ctx->slots, &ctx->units, &ctx->Lw_fb};
+    for (DevBuf* b : bufs)
+        if (b->p) cudaFree(b->p);
+    if (ctx->d_rec) cudaFree(ctx->d_rec);
+    if (ctx->d_w) cudaFree(ctx->d_w);
+    if (ctx->d_eye) cudaFree(ctx->d_eye);
+    if (ctx->d_ones) cudaFree(ctx->d_ones);
+    if (ctx->d_small) cudaFree(ctx->d_small);
+    if (ctx->h_small) cudaFreeHost(ctx->h_small);
+    if (ctx->h_stage) cudaFreeHost(ctx->h_stage);
+    for (cudaEvent_t e : ctx->ev_corr)
+        if (e) cudaEventDestroy(e);
+    if (ctx->own_stream && ctx->stream) cudaStreamDestroy(ctx->stream);
+    cudaGetLastError();
+    delete ctx;
+}
+
+dock_status dock_init(const dock_grid_desc* g, const float* receptor, const float* weights, dock_ctx** out)
+{
+    if (!out) return DOCK_E_INVALID_ARG;
+    *out = nullptr;
+    if (!g || !receptor || !weights) return DOCK_E_INVALID_ARG;
+    if (g->nx < 1 || g->ny < 1 || g->nz < 1 || g->n_terms < 1 || g->m_max < 1 || !(g->spacing > 0.f) ||
+        !std::isfinite(g->spacing))
+        return DOCK_E_INVALID_ARG;
+    if (g->n_terms > DOCK_MAX_TERMS || g->m_max > DOCK_MAX_M) return DOCK_E_UNSUPPORTED;
+    if ((int64_t)g->nx * g->ny * g->nz >= (int64_t(1) << 31) - 1) return DOCK_E_UNSUPPORTED;
+
+    dock_ctx* ctx = new (std::nothrow) dock_ctx();
+    if (!ctx) return DOCK_E_OOM;
+    ctx->device = g->device;
+    ctx->nx = g->nx;
+    ctx->ny = g->ny;
+    ctx->nz = g->nz;
+    ctx->P = g->n_terms;
+    ctx->m_max = g->m_max;
+    ctx->spacing = g->spacing;
+    auto bail = [&](dock_status s) {
+        dock_destroy(ctx);
+        return s;
+    };
+    if (cudaSetDevice(ctx->device) != cudaSuccess) {
+        cudaGetLastError();
+        return bail(DOCK_E_CUDA);
+    }
+    if (g->stream) {
+        ctx->stream = static_cast<cudaStream_t>(g->stream);
+    } else {
+        if (cudaStreamCreateWithFlags(&ctx->stream, cudaStreamNonBlocking) != cudaSuccess) return bail(DOCK_E_CUDA);
+        ctx->own_stream = true;
+    }
+    if (cudaEventCreate(&ctx->ev_corr[0]) != cudaSuccess || cudaEventCreate(&ctx->ev_corr[1]) != cudaSuccess)
+        return bail(DOCK_E_CUDA);
+    int v = 0;
+    if (cudaDeviceGetAttribute(&v, cudaDevAttrMultiProcessorCount, ctx->device) == cudaSuccess) ctx->n_sms = v;
+    if (cudaDeviceGetAttribute(&v, cudaDevAttrL2CacheSize, ctx->device) == cudaSuccess) ctx->l2_bytes = v;
+    ctx->geo = choose_geo(ctx->nx, ctx->ny, ctx->nz, ctx->m_max);
+    const dk::Geo& G = ctx->geo;
+    const int P = ctx->P;
+    const size_t n_in = (size_t)P * ctx->nx * ctx->ny * ctx->nz;
+    const size_t n_pad = (size_t)P * G.Xp * G.Yp * G.Zp;
+
+    // weights (host or device) -> host copy for validation
+    std::vector<float> w(P);
+    if (is_device_ptr(weights)) {
+        if (cudaMemcpy(w.data(), weights, sizeof(float) * P, cudaMemcpyDeviceToHost) != cudaSuccess)
+            return bail(DOCK_E_CUDA);
+    } else {
+        memcpy(w.data(), weights, sizeof(float) * P);
+    }
+    for (float x : w)
+        if (!std::isfinite(x)) return bail(DOCK_E_INVALID_ARG);
+
+    if (cudaMalloc(&ctx->d_rec, n_pad * sizeof(float)) != cudaSuccess) {
+        cudaGetLastError();
+        return bail(DOCK_E_OOM);
+    }
+    float* d_src = nullptr;
+    bool rec_dev = is_device_ptr(receptor);
+    if (rec_dev) {
+        d_src = const_cast<float*>(receptor);
+    } else {
+        for (size_t i = 0; i < n_in; i++)
+            if (!std::isfinite(receptor[i])) return bail(DOCK_E_INVALID_ARG);
+        if (cudaMalloc(&d_src, n_in * sizeof(float)) != cudaSuccess) {
+            cudaGetLastError();
+            return bail(DOCK_E_OOM);
+        }
+        if (cudaMemcpyAsync(d_src, receptor, n_in * sizeof(float), cudaMemcpyHostToDevice, ctx->stream) !=
+            cudaSuccess) {
+            cudaFree(d_src);
+            return bail(DOCK_E_CUDA);
+        }
+    }
+    bool ok = cudaMalloc(&ctx->d_small, 64) == cudaSuccess && cudaHostAlloc(&ctx->h_small, 64, 0) == cudaSuccess &&
+              cudaMalloc(&ctx->d_w, sizeof(float) * P) == cudaSuccess &&
+              cudaMalloc(&ctx->d_eye, sizeof(float) * P * P) == cudaSuccess &&
+              cudaMalloc(&ctx->d_ones, sizeof(float) * P) == cudaSuccess;
+    if (!ok) {
+        if (!rec_dev) cudaFree(d_src);
+        cudaGetLastError();
+        return bail(DOCK_E_OOM);
+    }
+    std::vector<float> eye((size_t)P * P, 0.f), ones(P, 1.f);
+    for (int p = 0; p < P; p++) eye[(size_t)p * P + p] = 1.f;
+    cudaMemcpy(ctx->d_w, w.data(), sizeof(float) * P, cudaMemcpyHostToDevice);
+    cudaMemcpy(ctx->d_eye, eye.data(), sizeof(float) * P * P, cudaMemcpyHostToDevice);
+    cudaMemcpy(ctx->d_ones, ones.data(), sizeof(float) * P, cudaMemcpyHostToDevice);
+    cudaMemsetAsync(ctx->d_small, 0, 64, ctx->stream);
+    if (rec_dev) {
+        dk::k_count_nonfinite<<<1024, 256, 0, ctx->stream>>>(d_src, n_in, reinterpret_cast<unsigned*>(ctx->d_small));
+    }
+    dk::k_pad_receptor<<<2048, 256, 0, ctx->stream>>>(d_src, ctx->d_rec, ctx->nx, ctx->ny, ctx->nz, G.Xp, G.Yp,
+                                                       G.Zp, P);
+    cudaError_t e = cudaGetLastError();
+    if (e == cudaSuccess) e = cudaMemcpyAsync(ctx->h_small, ctx->d_small, 16, cudaMemcpyDeviceToHost, ctx->stream);
+    if (e == cudaSuccess) e = cudaStreamSynchronize(ctx->stream);
+    if (!rec_dev) cudaFree(d_src);
+    if (e != cudaSuccess) return bail(DOCK_E_CUDA);
+    if (ctx->h_small[0] != 0) return bail(DOCK_E_INVALID_ARG);
+    for (int m = 1; m <= ctx->m_max; m++) {
+        dock_status s = make_plan(ctx, m);
+        if (s != DOCK_OK && m == ctx->m_max) return bail(s);
+    }
+    *out = ctx;
+    return DOCK_OK;
+}
+
+dock_status dock_set_tuning(dock_ctx* ctx, int key, int64_t value)
+{
+    if (!ctx) return DOCK_E_INVALID_ARG;
+    switch (key) {
+        case DOCK_TUNE_REGIONS:
+            if (value < 0) return fail(ctx, DOCK_E_INVALID_ARG, "regions < 0");
+            ctx->regions_override = (int)value;
+            return DOCK_OK;
+        case DOCK_TUNE_FORCE_FALLBACK: ctx->force_fallback = value ? 1 : 0; return DOCK_OK;
+        case DOCK_TUNE_CAND_CAP:
+            if (value < 32 || value > (1 << 20)) return fail(ctx, DOCK_E_INVALID_ARG, "cand cap out of range");
+            ctx->cand_cap = (int)value;
+            return DOCK_OK;
+    }
+    return fail(ctx, DOCK_E_INVALID_ARG, "unknown tuning key %d", key);
+}
+
+dock_status dock_get_info(const dock_ctx* ctx, dock_info* info)
+{
+    if (!ctx || !info) return DOCK_E_INVALID_ARG;
+    memset(info, 0, sizeof(*info));
+    info->lanes_x = ctx->geo.LX;
+    info->tile_x = ctx->geo.TX;
+    info->tile_y = ctx->geo.TY;
+    info->tile_z = ctx->geo.TZ;
+    info->n_tiles = ctx->geo.ntiles;
+    const MPlan& pl = ctx->plan[ctx->m_max];
+    info->n_stages = pl.nstage;
+    info->smem_bytes = pl.smem;
+    info->regions_last = ctx->regions_last;
+    info->items_last = ctx->items_last;
+    info->fallback_last = ctx->fallback_last;
+    info->cand_max_last = ctx->cand_max_last;
+    info->kernels_last = ctx->kernels_last;
+    info->rot_batch = dk::RB;
+    info->x_per_thread = dk::XT;
+    info->padded_x = ctx->geo.Xp;
+    info->padded_y = ctx->geo.Yp;
+    info->padded_z = ctx->geo.Zp;
+    info->l2_bytes = ctx->l2_bytes;
+    info->corr_ms_last = -1.0;
+    if (ctx->ev_corr_valid) {
+        float ms = 0.f;
+        if (cudaEventElapsedTime(&ms, ctx->ev_corr[0], ctx->ev_corr[1]) == cudaSuccess) info->corr_ms_last = ms;
+        else cudaGetLastError();
+    }
+    info->n_sms = ctx->n_sms;
+    return DOCK_OK;
+}
+
+dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n_probes, const double* rot,
+                             int n_rot, int64_t unit_begin, int64_t unit_end, int k, int rho, dock_pose* out)
+{
+    TRY(check_ctx(ctx));
+    ctx->kernels_last = 0;
+    ctx->ev_corr_valid = false;
+    if (!rot || !out || n_rot < 1) return fail(ctx, DOCK_E_INVALID_ARG, "null rotations/output or n_rot < 1");
+    if (k < 1) return fail(ctx, DOCK_E_INVALID_ARG, "k < 1");
+    if (k > DOCK_MAX_K) return fail(ctx, DOCK_E_UNSUPPORTED, "k > %d", DOCK_MAX_K);
+    if (rho < 0 || 2 * rho + 1 > std::min(ctx->nx, std::min(ctx->ny, ctx->nz)))
+        return fail(ctx, DOCK_E_INVALID_ARG, "rho out of range");
+    const double ball = std::pow(2.0 * rho + 1.0, 3);
+    if ((double)k * ball > (double)ctx->nx * ctx->ny * ctx->nz)
+        return fail(ctx, DOCK_E_INVALID_ARG, "k*(2rho+1)^3 exceeds the number of translations");
+    int m = 0;
+    TRY(validate_probes(ctx, probes, n_probes, &m));
+    if (unit_begin < 0 || unit_end < unit_begin || unit_end > (int64_t)n_probes * n_rot)
+        return fail(ctx, DOCK_E_INVALID_ARG, "bad unit range");
+    const int64_t n_units64 = unit_end - unit_begin;
+    if (n_units64 > (int64_t)1 << 28) return fail(ctx, DOCK_E_UNSUPPORTED, "too many units in one call");
+    const int n_units = (int)n_units64;
+    if (n_units == 0) return DOCK_OK;
+    TRY(make_plan(ctx, m));
+
+    const bool rot_dev = is_device_ptr(rot);
+    if (!rot_dev) {
+        for (int64_t i = 0; i < (int64_t)9 * n_rot; i++)
+            if (!std::isfinite(rot[i])) return fail(ctx, DOCK_E_INVALID_ARG, "non-finite rotation");
+    }
+    const double *d_xyz, *d_rot;
+    const float* d_coef;
+    const int* d_off;
+    TRY(stage_inputs(ctx, probes, n_probes, rot, n_rot, &d_xyz, &d_coef, &d_off, &d_rot));
+
+    const int P = ctx->P, m3 = m * m * m;
+    const int64_t n_batches = (n_units + dk::RB - 1) / dk::RB;
+    const int cap = ctx->cand_cap;
+    TRY(ensure(ctx, ctx->Lw, sizeof(float) * n_batches * P * m3 * dk::RB));
+    TRY(ensure(ctx, ctx->T, sizeof(unsigned long long) * n_units));
+    TRY(ensure(ctx, ctx->mu, sizeof(unsigned long long) * n_units));
+    TRY(ensure(ctx, ctx->cnt, sizeof(unsigned int) * n_units));
+    TRY(ensure(ctx, ctx->cand, sizeof(unsigned long long) * (size_t)n_units * cap));
+    TRY(ensure(ctx, ctx->fb_list, sizeof(int) * n_units));
+    const bool out_dev = is_device_ptr(out);
+    void* d_poses = out;
+    if (!out_dev) {
+        TRY(ensure(ctx, ctx->poses, sizeof(dock_pose) * (size_t)n_units * k));
+        d_poses = ctx->poses.p;
+    }
+
+    unsigned int* fb_cnt = reinterpret_cast<unsigned int*>(ctx->d_small + 1);
+    unsigned int* cand_max = reinterpret_cast<unsigned int*>(ctx->d_small + 2);
+    CU(cudaMemsetAsync(ctx->d_small, 0, 4, ctx->stream));
+    dk::k_reset<<<(n_units + 255) / 256, 256, 0, ctx->stream>>>(
+        static_cast<unsigned long long*>(ctx->T.p), static_cast<unsigned long long*>(ctx->mu.p),
+        static_cast<unsigned int*>(ctx->cnt.p), n_units, fb_cnt, cand_max);
+    CU(cudaGetLastError());
+    ctx->kernels_last++;
+
+    // a1: voxelize (+ rotation / box validation)
+    TRY(run_voxelize(ctx, m, n_units, unit_begin, nullptr, n_rot, d_xyz, d_coef, d_off, d_rot, ctx->d_w,
+                     static_cast<float*>(ctx->Lw.p)));
+
+    // a2-a5: correlation + fused weighted score + per-warp top-32 lists
+    const int G = choose_regions(ctx, n_batches);
+    dk::CorrArgs a = corr_args(ctx, m, n_units, G, static_cast<const float*>(ctx->Lw.p));
+    a.k = k;
+    a.rho = rho;
+    a.T = static_cast<unsigned long long*>(ctx->T.p);
+    a.mu = static_cast<unsigned long long*>(ctx->mu.p);
+    a.cnt = static_cast<unsigned int*>(ctx->cnt.p);
+    a.cand = static_cast<unsigned long long*>(ctx->cand.p);
+    a.cap = cap;
+    const int64_t items = n_batches * G;
+    if (items > 0x7fffffff) return fail(ctx, DOCK_E_UNSUPPORTED, "too many work items");
+    CU(cudaEventRecord(ctx->ev_corr[0], ctx->stream));
+    CU(launch_corr<false>(m, ctx->plan[m], a, (int)items, ctx->stream));
+    CU(cudaEventRecord(ctx->ev_corr[1], ctx->stream));
+    ctx->ev_corr_valid = true;
+    ctx->kernels_last++;
+    ctx->regions_last = G;
+    ctx->items_last = items;
+
+    // a6: per-rotation merge + greedy filter
+    dk::MergeArgs ma{};
+    ma.n_slots = n_units;
+    ma.k = k;
+    ma.rho = rho;
+    ma.cap = cap;
+    ma.n_rot = n_rot;
+    ma.nx = ctx->nx;
+    ma.ny = ctx->ny;
+    ma.nz = ctx->nz;
+    ma.unit_begin = unit_begin;
+    ma.cand = a.cand;
+    ma.cnt = a.cnt;
+    ma.mu = a.mu;
+    ma.force_fallback = ctx->force_fallback;
+    ma.poses = d_poses;
+    ma.fb_list = static_cast<int*>(ctx->fb_list.p);
+    ma.fb_cnt = fb_cnt;
+    ma.cand_max = cand_max;
+    dk::k_merge<<<(n_units + 7) / 8, 256, 0, ctx->stream>>>(ma);
+    CU(cudaGetLastError());
+    ctx->kernels_last++;
+
+    CU(cudaMemcpyAsync(ctx->h_small, ctx->d_small, 16, cudaMemcpyDeviceToHost, ctx->stream));
+    CU(cudaStreamSynchronize(ctx->stream));
+    TRY(check_status_word(ctx));
+    const int nfb = ctx->h_small[1];
+    ctx->fallback_last = nfb;
+    ctx->cand_max_last = (unsigned)ctx->h_small[2];
+    if (nfb > 0)
+        TRY(run_fallback(ctx, m, nfb, unit_begin, n_rot, d_xyz, d_coef, d_off, d_rot, k, rho, d_poses));
+    if (!out_dev)
+        CU(cudaMemcpyAsync(out, d_poses, sizeof(dock_pose) * (size_t)n_units * k, cudaMemcpyDeviceToHost,
+                           ctx->stream));
+    CU(cudaStreamSynchronize(ctx->stream));
+    return DOCK_OK;
+}
+
+dock_status dock_probe(dock_ctx* ctx, const dock_probe_desc* probe, const double* rot, int n_rot, int k, int rho,
+                       dock_pose* out)
+{
+    return dock_probe_batch(ctx, probe, 1, rot, n_rot, 0, n_rot, k, rho, out);
+}
+
+dock_status dock_score_grid(dock_ctx* ctx, const dock_probe_desc* probe, const double* rot9, float* out,
+                            float* per_term)
+{
+    TRY(check_ctx(ctx));
+    ctx->kernels_last = 0;
+    if (!rot9 || !out) return fail(ctx, DOCK_E_INVALID_ARG, "null rotation/output");
+    int m = 0;
+    TRY(validate_probes(ctx, probe, 1, &m));
+    TRY(make_plan(ctx, m));
+    const double *d_xyz, *d_rot;
+    const float* d_coef;
+    const int* d_off;
+    TRY(stage_inputs(ctx, probe, 1, rot9, 1, &d_xyz, &d_coef, &d_off, &d_rot));
+    const size_t ncell = (size_t)ctx->nx * ctx->ny * ctx->nz;
+    const int m3 = m * m * m;
+    TRY(ensure(ctx, ctx->Lw, sizeof(float) * ctx->P * m3 * dk::RB));
+    const bool out_dev = is_device_ptr(out);
+    const bool pt_dev = per_term && is_device_ptr(per_term);
+    size_t need = (out_dev ? 0 : ncell) + (per_term && !pt_dev ? ncell * ctx->P : 0);
+    if (need) TRY(ensure(ctx, ctx->grid, sizeof(float) * need));
+    float* g_out = out_dev ? out : static_cast<float*>(ctx->grid.p);
+    float* g_pt = per_term ? (pt_dev ? per_term : static_cast<float*>(ctx->grid.p) + (out_dev ? 0 : ncell)) : nullptr;
+    CU(cudaMemsetAsync(ctx->d_small, 0, 4, ctx->stream));
+    TRY(run_voxelize(ctx, m, 1, 0, nullptr, 1, d_xyz, d_coef, d_off, d_rot, ctx->d_w, static_cast<float*>(ctx->Lw.p)));
+    TRY(run_grid(ctx, m, 1, static_cast<const float*>(ctx->Lw.p), g_out));
+    if (per_term) {
+        for (int p = 0; p < ctx->P; p++) {
+            TRY(run_voxelize(ctx, m, 1, 0, nullptr, 1, d_xyz, d_coef, d_off, d_rot, ctx->d_eye + (size_t)p * ctx->P,
+                             static_cast<float*>(ctx->Lw.p)));
+            TRY(run_grid(ctx, m, 1, static_cast<const float*>(ctx->Lw.p), g_pt + ncell * p));
+        }
+    }
+    CU(cudaMemcpyAsync(ctx->h_small, ctx->d_small, 16, cudaMemcpyDeviceToHost, ctx->stream));
+    CU(cudaStreamSynchronize(ctx->stream));
+    TRY(check_status_word(ctx));
+    if (!out_dev) CU(cudaMemcpyAsync(out, g_out, sizeof(float) * ncell, cudaMemcpyDeviceToHost, ctx->stream));
+    if (per_term && !pt_dev)
+        CU(cudaMemcpyAsync(per_term, g_pt, sizeof(float) * ncell * ctx->P, cudaMemcpyDeviceToHost, ctx->stream));
+    CU(cudaStreamSynchronize(ctx->stream));
+    return DOCK_OK;
+}
+
+dock_status dock_voxelize(dock_ctx* ctx, const dock_probe_desc* probe, const double* rot, int n_rot, float* out)
+{
+    TRY(check_ctx(ctx));
+    ctx->kernels_last = 0;
+    ctx->ev_corr_valid = false;
+    if (!rot || !out || n_rot < 1) return fail(ctx, DOCK_E_INVALID_ARG, "null rotation/output");
+    int m = 0;
+    TRY(validate_probes(ctx, probe, 1, &m));
+    const double *d_xyz, *d_rot;
+    const float* d_coef;
+    const int* d_off;
+    TRY(stage_inputs(ctx, probe, 1, rot, n_rot, &d_xyz, &d_coef, &d_off, &d_rot));
+    const int m3 = m * m * m, P = ctx->P;
+    const int64_t nb = (n_rot + dk::RB - 1) / dk::RB;
+    TRY(ensure(ctx, ctx->Lw, sizeof(float) * nb * P * m3 * dk::RB));
+    const bool out_dev = is_device_ptr(out);
+    const size_t n_out = (size_t)n_rot * P * m3;
+    if (!out_dev) TRY(ensure(ctx, ctx->grid, sizeof(float) * n_out));
+    float* g_out = out_dev ? out : static_cast<float*>(ctx->grid.p);
+    CU(cudaMemsetAsync(ctx->d_small, 0, 4, ctx->stream));
+    TRY(run_voxelize(ctx, m, n_rot, 0, nullptr, n_rot, d_xyz, d_coef, d_off, d_rot, ctx->d_ones,
+                     static_cast<float*>(ctx->Lw.p)));
+    int n = (int)n_out;
+    dk::k_unpack_L<<<(n + 255) / 256, 256, 0, ctx->stream>>>(static_cast<const float*>(ctx->Lw.p), g_out, n_rot, P,
+                                                              m3);
+    CU(cudaGetLastError());
+    CU(cudaMemcpyAsync(ctx->h_small, ctx->d_small, 16, cudaMemcpyDeviceToHost, ctx->stream));
+    CU(cudaStreamSynchronize(ctx->stream));
+    TRY(check_status_word(ctx));
+    if (!out_dev) CU(cudaMemcpyAsync(out, g_out, sizeof(float) * n_out, cudaMemcpyDeviceToHost, ctx->stream));
+    CU(cudaStreamSynchronize(ctx->stream));
+    return DOCK_OK;
+}
+
+}  // extern "C"

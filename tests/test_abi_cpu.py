@@ -1,0 +1,74 @@
+"""CPU-only checks of the boundary: libdock.so builds for sm_100a, loads, and exports every
+symbol include/dock.h declares; the binding fails loudly without the library; no compute."""
+import ctypes
+import os
+import re
+
+import pytest
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+
+
+@pytest.fixture(scope="module")
+def lib():
+    from paper_conf_ipps_sukhwanih10_b200 import build
+    build.build_native()
+    from paper_conf_ipps_sukhwanih10_b200 import _native
+    return _native.lib()
+
+
+def _header_functions():
+    src = open(os.path.join(ROOT, "include", "dock.h")).read()
+    src = re.sub(r"/\*.*?\*/", "", src, flags=re.S)
+    return sorted(set(re.findall(r"\b(dock_[a-z_]+)\s*\(", src)))
+
+
+def test_header_symbols_exported(lib):
+    names = _header_functions()
+    assert "dock_init" in names and "dock_probe_batch" in names
+    for n in names:
+        assert hasattr(lib, n), f"libdock.so does not export {n}"
+    from paper_conf_ipps_sukhwanih10_b200 import _native
+    assert sorted(_native.EXPORTS) == names
+
+
+def test_status_strings(lib):
+    for code, name in [(0, b"DOCK_OK"), (-1, b"DOCK_E_INVALID_ARG"), (-3, b"DOCK_E_PROBE_OUTSIDE_GRID"),
+                       (-4, b"DOCK_E_BAD_ROTATION"), (-5, b"DOCK_E_CUDA")]:
+        assert lib.dock_status_string(code) == name
+
+
+def test_null_arguments_rejected_without_gpu(lib):
+    out = ctypes.c_void_p()
+    assert lib.dock_init(None, None, None, ctypes.byref(out)) == -1
+    assert lib.dock_probe_batch(None, None, 0, None, 0, 0, 0, 1, 0, None) == -1
+    lib.dock_destroy(None)
+
+
+def test_struct_layouts():
+    from paper_conf_ipps_sukhwanih10_b200 import _native as N
+    assert ctypes.sizeof(N.dock_pose) == 16
+    assert ctypes.sizeof(N.dock_probe_desc) == 24
+    assert ctypes.sizeof(N.dock_grid_desc) == 40
+
+
+def test_sass_is_sm100a_with_tma():
+    """The hot kernel is compiled for sm_100a and issues TMA (UTMALDG) + bulk copies (UBLKCP)."""
+    import shutil
+    import subprocess
+    from paper_conf_ipps_sukhwanih10_b200 import build
+    lib_path = build.build_native()
+    cuobjdump = shutil.which("cuobjdump") or "/usr/local/cuda/bin/cuobjdump"
+    if not os.path.exists(cuobjdump) and not shutil.which("cuobjdump"):
+        pytest.skip("cuobjdump not available")
+    out = subprocess.run([cuobjdump, "-sass", lib_path], capture_output=True, text=True).stdout
+    assert "sm_100a" in out
+    assert "UTMALDG" in out and "UBLKCP" in out and "FFMA" in out
+
+
+def test_missing_library_fails_loudly(monkeypatch, tmp_path):
+    from paper_conf_ipps_sukhwanih10_b200 import _native
+    monkeypatch.setattr(_native, "_lib", None)
+    monkeypatch.setattr(_native, "LIB_PATH", str(tmp_path / "nope.so"))
+    with pytest.raises(ImportError):
+        _native.lib()

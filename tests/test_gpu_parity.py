@@ -1,0 +1,312 @@
+"""GPU parity: the CUDA path (through the C ABI) against the FP64 oracle.
+
+Bars: voxel indices bit-exact; score grids |S_gpu - S_orc| <= 1e-4 * A;
+integer-valued inputs bitwise; poses validated tie-aware (tests/validator.py); results
+invariant (bitwise) to batch position, batch size, launch configuration and shard range.
+"""
+import concurrent.futures as cf
+
+import numpy as np
+import pytest
+
+import dockgen as g
+from validator import validate_unit
+
+pytestmark = pytest.mark.gpu
+H = g.SPACING
+
+
+@pytest.fixture(scope="module")
+def D():
+    import torch
+    assert torch.cuda.is_available(), "GPU tests need a CUDA device"
+    from paper_conf_ipps_sukhwanih10_b200 import build
+    build.build_native()
+    import paper_conf_ipps_sukhwanih10_b200 as D
+    return D
+
+
+def _oracle_SA(orc, R, w, pr, q):
+    L = orc.voxelize(pr.xyz, pr.coef, pr.m, q, H)
+    return orc.score_grid(R, L, w)
+
+
+def _oracle_units(orc, R, w, probes, rot, units, threads=8):
+    def one(u):
+        pr, r = probes[u // len(rot)], u % len(rot)
+        return _oracle_SA(orc, R, w, pr, rot[r])
+    with cf.ThreadPoolExecutor(threads) as ex:
+        return list(ex.map(one, units))
+
+
+# ----------------------------------------------------------------------------- voxelize
+
+
+@pytest.mark.parametrize("m", [1, 2, 3, 4, 5, 8])
+def test_voxelize_matches_oracle(D, orc, m):
+    P = 3
+    R = g.receptor_uniform((16, 16, 16), P)
+    ctx = D.dock_init(R, g.weights(P), H, m_max=8)
+    rot = g.rotations(40, with_cube_group=True)
+    for i in range(3):
+        pr = g.probe(i, m, P) if m > 1 else g.Probe(np.zeros((1, 3)), np.ones((1, P), np.float32), 1)
+        Lg = D.dock_voxelize(ctx, pr, rot)
+        for r in range(rot.shape[0]):
+            Lo = orc.voxelize(pr.xyz, pr.coef, m, rot[r], H)
+            assert np.array_equal(Lg[r] != 0, Lo != 0)
+            assert np.allclose(Lg[r], Lo, rtol=1e-6, atol=1e-6)
+    ctx.close()
+
+
+# ----------------------------------------------------------------------------- score grids
+
+
+@pytest.mark.parametrize("shape,m,P,kind", [
+    ((128, 12, 10), 4, 4, "ftmap"),     # lanes_x = 16 path, ragged y/z tiles
+    ((64, 20, 11), 5, 4, "uniform"),    # lanes_x = 8 path
+    ((37, 13, 9), 4, 2, "uniform"),     # lanes_x = 4 path, ragged everywhere
+    ((40, 24, 24), 8, 3, "uniform"),    # largest probe grid
+    ((33, 17, 19), 1, 1, "uniform"),    # m = 1
+])
+def test_score_grid_within_tolerance(D, orc, shape, m, P, kind):
+    R = g.receptor(kind, shape, P)
+    w = g.weights(P)
+    ctx = D.dock_init(R, w, H, m_max=m)
+    rot = g.rotations(4)
+    for i, q in enumerate(rot):
+        pr = g.probe(i + 1, m, P) if m > 1 else g.Probe(np.zeros((1, 3)), np.ones((1, P), np.float32), 1)
+        S_g, C_g = D.dock_score_grid(ctx, pr, q, per_term=True)
+        S_o, A_o = _oracle_SA(orc, R, w, pr, q)
+        err = np.abs(S_g.astype(np.float64) - S_o)
+        assert (err <= 1e-4 * A_o + 1e-12).all(), f"max err/A {np.max(err / np.maximum(A_o, 1e-30))}"
+        # per-term grids are the unweighted C_p: S = sum_p w_p C_p (reading Q6)
+        L = orc.voxelize(pr.xyz, pr.coef, m, q, H)
+        for p in range(P):
+            e = np.eye(P, dtype=np.float32)[p]
+            Cp, Ap = orc.score_grid(R, L, e)
+            assert (np.abs(C_g[p] - Cp) <= 1e-4 * Ap + 1e-12).all()
+    ctx.close()
+
+
+def test_delta_probe_bitwise(D):
+    """P4: one atom at the centre, m = 1, coef = e_p -> S == R_p bitwise on the GPU."""
+    P = 3
+    R = g.receptor_uniform((40, 18, 12), P)
+    ctx = D.dock_init(R, np.ones(P, np.float32), H, m_max=1)
+    for p in range(P):
+        coef = np.zeros((1, P), np.float32)
+        coef[0, p] = 1
+        S = D.dock_score_grid(ctx, g.Probe(np.zeros((1, 3)), coef, 1), np.eye(3).reshape(9))
+        assert np.array_equal(S, R[p])
+    ctx.close()
+
+
+def test_shift_equivariance_bitwise(D):
+    """P5: single atom on voxel v0 -> S = roll(R, -v0) bitwise."""
+    R = g.receptor_uniform((24, 20, 16), 1)
+    ctx = D.dock_init(R, np.ones(1, np.float32), H, m_max=4)
+    for v0 in [(0, 0, 0), (3, 1, 2), (1, 3, 3)]:
+        pr = g.voxel_centre_probe([v0], 4, 1)
+        S = D.dock_score_grid(ctx, pr, np.eye(3).reshape(9))
+        assert np.array_equal(S, np.roll(R[0], (-v0[2], -v0[1], -v0[0]), axis=(0, 1, 2)))
+    ctx.close()
+
+
+def test_integer_inputs_bitwise_grid(D, orc):
+    """P9: integer-valued inputs -> the FP32 score grid equals the FP64 oracle exactly."""
+    P, m = 4, 4
+    R = g.receptor_integer((48, 20, 18), P)
+    w = g.weights_integer(P)
+    ctx = D.dock_init(R, w, H, m_max=m)
+    rot = g.rotations(3, with_cube_group=True)[:6]
+    for i, q in enumerate(rot):
+        pr = g.probe(i, m, P, integer=True)
+        S_g = D.dock_score_grid(ctx, pr, q)
+        S_o, _ = _oracle_SA(orc, R, w, pr, q)
+        assert np.array_equal(S_g.astype(np.float64), S_o)
+    ctx.close()
+
+
+# ----------------------------------------------------------------------------- poses
+
+
+def _dock_and_validate(D, orc, R, w, probes, rot, k, rho, units=None, **tune):
+    ctx = D.dock_init(R, w, H, m_max=max(p.m for p in probes))
+    for key, v in tune.items():
+        D.dock_set_tuning(ctx, key, v)
+    poses = D.dock_probe_batch(ctx, probes, rot, k=k, rho=rho)
+    info = D.dock_get_info(ctx)
+    ctx.close()
+    n_units = len(probes) * len(rot)
+    units = list(range(n_units)) if units is None else units
+    SA = _oracle_units(orc, R, w, probes, rot, units)
+    mism = 0
+    for u, (S, A) in zip(units, SA):
+        assert (poses[u]["rot"] == u % len(rot)).all()
+        mism += validate_unit(S, A, poses[u]["t_lin"], poses[u]["score"], k, rho)
+    return poses, info, mism
+
+
+@pytest.mark.parametrize("rho,k", [(0, 1), (0, 4), (1, 1), (1, 4), (2, 3)])
+def test_poses_toy_config(D, orc, rho, k):
+    c = g.CONFIGS["toy"]
+    R = g.receptor_ftmap_like(c.n, c.P)
+    w = g.weights(c.P)
+    probes = g.probes(2, c.m, c.P)
+    rot = g.rotations(c.n_rot, with_cube_group=True)
+    _dock_and_validate(D, orc, R, w, probes, rot, k, rho)
+
+
+@pytest.mark.parametrize("kind", ["ftmap", "uniform"])
+@pytest.mark.parametrize("rho", [0, 1])
+def test_poses_mid_config(D, orc, kind, rho):
+    P, m = 4, 4
+    R = g.receptor(kind, (48, 40, 36), P)
+    w = g.weights(P)
+    probes = g.probes(3, m, P)
+    rot = g.rotations(21)
+    _, info, mism = _dock_and_validate(D, orc, R, w, probes, rot, 4, rho)
+    assert info["fallback_last"] <= 2
+
+
+@pytest.mark.parametrize("rho,k", [(0, 4), (1, 4), (0, 1)])
+def test_integer_inputs_exact_poses(D, orc, rho, k):
+    """P9: integer inputs -> poses (t_lin and score) equal the oracle exactly, ties included."""
+    P, m = 4, 3
+    R = g.receptor_integer((40, 24, 20), P, lo=-2, hi=2)
+    w = g.weights_integer(P)
+    probes = g.probes(2, m, P, integer=True)
+    rot = g.rotations(10)
+    ctx = D.dock_init(R, w, H, m_max=m)
+    poses = D.dock_probe_batch(ctx, probes, rot, k=k, rho=rho)
+    ctx.close()
+    t_o, s_o, st = orc.dock(R, w, H, probes, rot, k, rho)
+    assert (st == 0).all()
+    assert np.array_equal(poses["t_lin"], t_o.astype(np.int32))
+    assert np.array_equal(poses["score"].astype(np.float64), s_o)
+
+
+def test_fallback_path_identical(D):
+    """The exact full-grid fallback returns the same poses (bitwise) as the candidate path."""
+    P, m = 4, 4
+    R = g.receptor_ftmap_like((48, 40, 36), P)
+    w = g.weights(P)
+    probes = g.probes(2, m, P)
+    rot = g.rotations(13)
+    ctx = D.dock_init(R, w, H, m_max=m)
+    for rho in (0, 1):
+        a = D.dock_probe_batch(ctx, probes, rot, k=4, rho=rho)
+        D.dock_set_tuning(ctx, D.DOCK_TUNE_FORCE_FALLBACK, 1)
+        b = D.dock_probe_batch(ctx, probes, rot, k=4, rho=rho)
+        assert D.dock_get_info(ctx)["fallback_last"] == len(probes) * len(rot)
+        D.dock_set_tuning(ctx, D.DOCK_TUNE_FORCE_FALLBACK, 0)
+        assert np.array_equal(a["t_lin"], b["t_lin"])
+        assert np.array_equal(a["score"].view(np.uint32), b["score"].view(np.uint32))
+        assert (b["flags"] & D.DOCK_POSE_FALLBACK).all()
+    ctx.close()
+
+
+def test_invariance_batch_shard_launch(D):
+    """Per-rotation results are bitwise independent of batch position, batch size,
+    regions per batch (launch configuration), candidate cap and shard range."""
+    P, m = 4, 4
+    R = g.receptor_ftmap_like((64, 48, 40), P)
+    w = g.weights(P)
+    probes = g.probes(3, m, P)
+    rot = g.rotations(19)
+    ctx = D.dock_init(R, w, H, m_max=m)
+    ref = D.dock_probe_batch(ctx, probes, rot, k=4, rho=1)
+    n = len(probes) * len(rot)
+    for b, e in [(0, 5), (5, 31), (31, n), (7, 8)]:
+        part = D.dock_probe_batch(ctx, probes, rot, unit_begin=b, unit_end=e, k=4, rho=1)
+        assert np.array_equal(part, ref[b:e])
+    for G in (1, 3, 7):
+        D.dock_set_tuning(ctx, D.DOCK_TUNE_REGIONS, G)
+        assert np.array_equal(D.dock_probe_batch(ctx, probes, rot, k=4, rho=1), ref)
+    D.dock_set_tuning(ctx, D.DOCK_TUNE_REGIONS, 0)
+    D.dock_set_tuning(ctx, D.DOCK_TUNE_CAND_CAP, 32)
+    assert np.array_equal(D.dock_probe_batch(ctx, probes, rot, k=4, rho=1)["t_lin"], ref["t_lin"])
+    D.dock_set_tuning(ctx, D.DOCK_TUNE_CAND_CAP, 1024)
+    # reversed rotation order: per-rotation results follow the rotation
+    rev = rot[::-1].copy()
+    out = D.dock_probe_batch(ctx, probes, rev, k=4, rho=1)
+    for pi in range(len(probes)):
+        for i in range(len(rot)):
+            a = out[pi * len(rot) + i]
+            b = ref[pi * len(rot) + len(rot) - 1 - i]
+            assert np.array_equal(a["t_lin"], b["t_lin"]) and np.array_equal(a["score"], b["score"])
+    ctx.close()
+
+
+def test_device_resident_io(D):
+    """Device-resident inputs/outputs (torch CUDA tensors) give the same poses as host I/O."""
+    import torch
+    P, m = 4, 4
+    R = g.receptor_ftmap_like((40, 32, 32), P)
+    w = g.weights(P)
+    probes = g.probes(2, m, P)
+    rot = g.rotations(9)
+    ctx = D.dock_init(torch.from_numpy(R).cuda(), torch.from_numpy(w).cuda(), H, m_max=m)
+    host = D.dock_probe_batch(ctx, probes, rot, k=4, rho=1)
+    dprobes = [{"xyz": torch.from_numpy(p.xyz).cuda(), "coef": torch.from_numpy(p.coef).cuda(), "m": p.m}
+               for p in probes]
+    out = torch.empty((len(probes) * len(rot), 4, 4), dtype=torch.int32, device="cuda")
+    D.dock_probe_batch(ctx, dprobes, torch.from_numpy(rot).cuda(), k=4, rho=1, out=out)
+    torch.cuda.synchronize()
+    assert np.array_equal(D.poses_from_device(out), host)
+    ctx.close()
+
+
+def test_errors(D):
+    P = 1
+    R = g.receptor_uniform((16, 16, 16), P)
+    ctx = D.dock_init(R, np.ones(P, np.float32), H, m_max=4)
+    pr = g.probe(0, 4, P)
+    with pytest.raises(D.DockError) as e:
+        D.dock_probe(ctx, pr, np.diag([1.0, 1.0, -1.0]).reshape(1, 9), k=1, rho=0)
+    assert e.value.status == -4
+    far = g.Probe(np.array([[4.0, 0, 0]]), np.ones((1, 1), np.float32), 4)
+    with pytest.raises(D.DockError) as e:
+        D.dock_probe(ctx, far, g.rotations(3), k=1, rho=0)
+    assert e.value.status == -3
+    with pytest.raises(D.DockError) as e:
+        D.dock_probe(ctx, pr, g.rotations(3), k=0, rho=0)
+    assert e.value.status == -1
+    with pytest.raises(D.DockError) as e:
+        D.dock_probe(ctx, pr, g.rotations(3), k=1, rho=8)
+    assert e.value.status == -1
+    with pytest.raises(D.DockError) as e:
+        D.dock_probe(ctx, g.probe(0, 5, P), g.rotations(3), k=1, rho=0)
+    assert e.value.status == -2
+    # the context is still usable after argument errors
+    D.dock_probe(ctx, pr, g.rotations(3), k=2, rho=1)
+    ctx.close()
+    with pytest.raises(D.DockError):
+        D.dock_init(np.full((1, 8, 8, 8), np.nan, np.float32), np.ones(1, np.float32), H, m_max=2)
+
+
+# ----------------------------------------------------------------------------- BASELINE configs
+
+
+def test_c64_config_sampled(D, orc):
+    """configs[1]: 64^3, 5^3 probe, 4 terms, 500 rotations, k=4 -- full GPU run, oracle on a sample."""
+    c = g.CONFIGS["c64"]
+    R = g.receptor_ftmap_like(c.n, c.P)
+    w = g.weights(c.P)
+    probes = g.probes(1, c.m, c.P)
+    rot = g.rotations(c.n_rot)
+    units = list(range(0, 500, 25)) + [1, 2, 3, 499]
+    _dock_and_validate(D, orc, R, w, probes, rot, c.k, 1, units=units)
+
+
+def test_prod_config_sampled(D, orc):
+    """configs[2] (the bench workload, same launch as bench.py): 128^3, 16 probes x 500 rotations,
+    k=4, rho=1 -- every unit docked on the GPU, a spread sample validated against the oracle."""
+    c = g.CONFIGS["prod"]
+    R = g.receptor_ftmap_like(c.n, c.P)
+    w = g.weights(c.P)
+    probes = g.probes(c.n_probes, c.m, c.P)
+    rot = g.rotations(c.n_rot)
+    units = [0, 1, 499, 500, 3777, 7999] + list(range(137, 8000, 811))
+    _, info, _ = _dock_and_validate(D, orc, R, w, probes, rot, c.k, 1, units=units)
+    assert info["fallback_last"] <= 80
