@@ -165,7 +165,7 @@ def _offsets(cut_vox: int) -> np.ndarray:
     return np.stack([ox.ravel(), oy.ravel(), oz.ravel()], axis=1)
 
 
-def _splat(prot: Protein, n: Sequence[int], spacing: float, cutoff: float, chunk: int = 64):
+def _splat(prot: Protein, n: Sequence[int], spacing: float, cutoff: float, chunk: int = 192):
     """Yield (flat voxel index, distance Å, atom index) for voxel/atom pairs with d < cutoff.
 
     Voxel (i, j, k) has its centre at (i, j, k) * spacing; indices wrap cyclically
@@ -174,6 +174,8 @@ def _splat(prot: Protein, n: Sequence[int], spacing: float, cutoff: float, chunk
     nx, ny, nz = n
     cv = int(math.ceil(cutoff / spacing)) + 1
     off = _offsets(cv)
+    # only offsets that can reach within the cutoff of an atom inside its base voxel
+    off = off[np.linalg.norm(off, axis=1) * spacing <= cutoff + spacing * math.sqrt(3.0)]
     base = np.floor(prot.xyz / spacing).astype(np.int64)
     for a0 in range(0, len(prot.xyz), chunk):
         a1 = min(len(prot.xyz), a0 + chunk)

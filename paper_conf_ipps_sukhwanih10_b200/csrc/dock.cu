@@ -393,7 +393,7 @@ dock_status run_voxelize(dock_ctx* ctx, int m, int n_slots, int64_t unit_begin, 
     v.spacing = ctx->spacing;
     v.Lw = Lw;
     v.status = ctx->d_small;
-    int n = n_slots * ctx->P;
+    int n = (n_slots + dk::RB - 1) / dk::RB * dk::RB * ctx->P;
     dk::k_voxelize<<<(n + 127) / 128, 128, 0, ctx->stream>>>(v);
     CU(cudaGetLastError());
     ctx->kernels_last++;
@@ -412,6 +412,7 @@ dk::CorrArgs corr_args(dock_ctx* ctx, int m, int n_slots, int G, const float* Lw
     a.tiles_per_region = (ctx->geo.ntiles + G - 1) / G;
     a.nstage = pl.nstage;
     a.stage_rec_bytes = pl.stage_rec_bytes;
+    a.box_bytes = pl.TXB * pl.TYB * pl.TZB * 4;
     a.stage_bytes = pl.stage_bytes;
     a.TXB = pl.TXB;
     a.TYB = pl.TYB;

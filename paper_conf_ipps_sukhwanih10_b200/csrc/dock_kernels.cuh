@@ -46,7 +46,8 @@ struct CorrArgs {
     int G;                      // regions per rotation batch
     int tiles_per_region;
     int nstage;
-    int stage_rec_bytes;        // TXB*TYB*TZB*4, multiple of 128
+    int stage_rec_bytes;        // TXB*TYB*TZB*4 rounded up to a multiple of 128 (stage offset)
+    int box_bytes;              // TXB*TYB*TZB*4 exactly (TMA transaction bytes)
     int stage_bytes;            // stage_rec_bytes + M^3*RB*4 (multiple of 128)
     int TXB, TYB, TZB;          // receptor box extents for this M
     // top-k mode
@@ -143,15 +144,27 @@ __device__ __forceinline__ void mbar_arrive(uint64_t* bar)
 {
     asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(smem_u32(bar)) : "memory");
 }
+__device__ __forceinline__ bool mbar_try_wait(uint64_t* bar, unsigned parity)
+{
+    uint32_t ok;
+    asm volatile(
+        "{\n\t.reg .pred p;\n\t"
+        "mbarrier.try_wait.parity.shared::cta.b64 p, [%1], %2;\n\t"
+        "selp.u32 %0, 1, 0, p;\n}\n"
+        : "=r"(ok)
+        : "r"(smem_u32(bar)), "r"(parity)
+        : "memory");
+    return ok != 0;
+}
+// Wait for the phase with the given parity.  A watchdog turns a lost transaction (which
+// would otherwise hang the GPU) into a trapped launch error after ~2^35 cycles (~17 s).
 __device__ __forceinline__ void mbar_wait(uint64_t* bar, unsigned parity)
 {
-    asm volatile(
-        "{\n\t.reg .pred p;\n"
-        "WAIT_%=:\n\t"
-        "mbarrier.try_wait.parity.shared::cta.b64 p, [%0], %1;\n\t"
-        "@!p bra WAIT_%=;\n}\n" ::"r"(smem_u32(bar)),
-        "r"(parity)
-        : "memory");
+    if (mbar_try_wait(bar, parity)) return;
+    const long long t0 = clock64();
+    while (!mbar_try_wait(bar, parity)) {
+        if (clock64() - t0 > (1ll << 35)) __trap();
+    }
 }
 __device__ __forceinline__ void tma_load_4d(void* dst, const CUtensorMap* map, int x, int y, int z, int c,
                                             uint64_t* bar)
@@ -225,14 +238,16 @@ struct VoxArgs {
 __global__ void k_voxelize(VoxArgs a)
 {
     int idx = blockIdx.x * blockDim.x + threadIdx.x;
-    if (idx >= a.n_slots * a.P) return;
+    const int n_pad = (a.n_slots + RB - 1) / RB * RB;   // the last batch is zero-padded
+    if (idx >= n_pad * a.P) return;
     int slot = idx / a.P, p = idx % a.P;
-    long long unit = a.unit_list ? static_cast<long long>(a.unit_list[slot]) : a.unit_begin + slot;
-    int probe = static_cast<int>(unit / a.n_rot), r = static_cast<int>(unit % a.n_rot);
-    const double* q = a.rot + 9 * static_cast<size_t>(r);
     const int m = a.m, m3 = m * m * m;
     float* dst = a.Lw + (static_cast<size_t>(slot / RB) * a.P + p) * m3 * RB + (slot % RB);
     for (int v = 0; v < m3; v++) dst[v * RB] = 0.0f;
+    if (slot >= a.n_slots) return;
+    long long unit = a.unit_list ? static_cast<long long>(a.unit_list[slot]) : a.unit_begin + slot;
+    int probe = static_cast<int>(unit / a.n_rot), r = static_cast<int>(unit % a.n_rot);
+    const double* q = a.rot + 9 * static_cast<size_t>(r);
 
     if (p == 0) {   // rotation check: |Q^T Q - I| <= 1e-9 and det > 0 (reading Q5)
         bool ok = true;
@@ -341,7 +356,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr(const __grid_constant__ CU
                 const int p = it % a.P;
                 const int tx = tile % a.g.ntx, ty = (tile / a.g.ntx) % a.g.nty, tz = tile / (a.g.ntx * a.g.nty);
                 unsigned char* st = smem + static_cast<size_t>(s) * a.stage_bytes;
-                mbar_arrive_expect_tx(&full[s], a.stage_rec_bytes + wbytes);
+                mbar_arrive_expect_tx(&full[s], a.box_bytes + wbytes);
                 tma_load_4d(st, &tmap, tx * a.g.TX, ty * a.g.TY, tz * a.g.TZ, p, &full[s]);
                 bulk_load(st + a.stage_rec_bytes, wsrc + static_cast<size_t>(p) * M3 * RB, wbytes, &full[s]);
             }
