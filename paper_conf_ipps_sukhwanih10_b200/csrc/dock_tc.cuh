@@ -1,0 +1,399 @@
+// dock_tc.cuh -- tensor-core (tcgen05) engine of the multi-term direct correlation
+// (north star (b): "Tensor cores are used only if an implicit-GEMM
+// form over the term channels meets the stated tolerance").
+//
+// Implicit GEMM per (rotation block, translation row):
+//   D[r][x] = sum_K A[r][K] * B[x][K],   r = 128 rotations (MMA M), x = 128 translations
+//   along one receptor x-row (MMA N), K = (channel group g, pass, vz, vy, vx, 8 "channels").
+// bf16x3 split keeps FP32-level accuracy (|err| ~ 1e-5 * A, tolerance 1e-4 * A, reading Q16):
+//   receptor voxel = 8 bf16 (Rhi_0..3, Rlo_0..3) of 4 channels, 16 B;
+//   pass 0 weights = (Whi_0..3, Whi_0..3)  -> Rhi*Whi + Rlo*Whi,
+//   pass 1 weights = (Wlo_0..3, 0, 0, 0, 0) -> Rhi*Wlo.
+// B needs no im2col: the receptor tile is stored [z][y][x][8 bf16] in shared memory, so the
+// K-major no-swizzle UMMA layout (core matrix = 8 rows x 16 B, rows 16 B apart, SBO = 128 B)
+// of "128 consecutive translations x (voxel vx, vx+1)" is the tile itself read at a start
+// address offset of the filter offset (vz, vy, vx); LBO = 16 B steps to voxel vx+1.
+// A (weights, K-major) streams through an 8-stage mbarrier ring (4 KB per K-step) and is
+// reused by the Q translation rows of a tile; D lives in TMEM (Q x 128 columns per buffer).
+// Epilogue: one thread per (rotation, half of the rows) reads its TMEM lane with
+// tcgen05.ld and keeps an exact per-thread top-LIST key list (no score grid in HBM),
+// published at item end exactly like the FFMA engine (k_merge is shared).
+#pragma once
+#include "dock_kernels.cuh"
+
+namespace tc {
+
+using dk::KEY_MAX;
+
+constexpr int ROT = 128;        // rotations per block (MMA M)
+constexpr int NT = 128;         // translations per row (MMA N)
+constexpr int NEPI = 8;         // epilogue warps (2 per TMEM lane quarter)
+constexpr int NTHREADS = (2 + NEPI) * 32;
+constexpr int WSTAGES = 8;      // weight ring depth
+constexpr int WCHUNK = 2 * ROT * 16;   // bytes of one K-step of A (2 K-chunks x 128 rotations x 16 B)
+constexpr int LIST = 16;        // per-thread candidate list
+
+struct TcArgs {
+    int nx, ny, nz;
+    int ntx, nty, ntz, ntiles;  // tiles: 128 x Q rows (y) x 1 (z)
+    int G_ch;                   // channel groups of 4
+    int n_slots, G, tiles_per_region;
+    int nsteps;
+    const unsigned char* W;     // [block][step][WCHUNK]
+    int TXB, TYB, TZB;
+    int box_bytes;              // one channel group's receptor box
+    int rec_stage_bytes;        // G_ch * box_bytes rounded to 1024
+    int n_rec_stages;           // 1 or 2
+    // top-k
+    int k, rho, cap;
+    unsigned long long* T;
+    unsigned long long* mu;
+    unsigned int* cnt;
+    unsigned long long* cand;
+    // grid mode
+    float* grid;
+};
+
+__device__ __forceinline__ uint64_t umma_desc(uint32_t saddr, uint32_t lbo, uint32_t sbo)
+{
+    uint64_t d = 0;
+    d |= static_cast<uint64_t>((saddr >> 4) & 0x3FFFu);
+    d |= static_cast<uint64_t>((lbo >> 4) & 0x3FFFu) << 16;
+    d |= static_cast<uint64_t>((sbo >> 4) & 0x3FFFu) << 32;
+    d |= static_cast<uint64_t>(1) << 46;   // descriptor version 1 (sm_100); no swizzle, base offset 0
+    return d;
+}
+
+// kind::f16 instruction descriptor: D f32, A/B bf16, both K-major, M x N.
+__host__ __device__ constexpr uint32_t umma_idesc(int m, int n)
+{
+    return (1u << 4) | (1u << 7) | (1u << 10) | (static_cast<uint32_t>(n >> 3) << 17) |
+           (static_cast<uint32_t>(m >> 4) << 24);
+}
+
+__device__ __forceinline__ void umma_bf16(uint32_t d_tmem, uint64_t a, uint64_t b, uint32_t idesc, uint32_t acc)
+{
+    asm volatile(
+        "{\n\t.reg .pred p;\n\tsetp.ne.b32 p, %4, 0;\n\t"
+        "tcgen05.mma.cta_group::1.kind::f16 [%0], %1, %2, %3, p;\n\t}\n" ::"r"(d_tmem),
+        "l"(a), "l"(b), "r"(idesc), "r"(acc)
+        : "memory");
+}
+__device__ __forceinline__ void umma_commit(uint64_t* bar)
+{
+    asm volatile("tcgen05.commit.cta_group::1.mbarrier::arrive::one.shared::cluster.b64 [%0];" ::"r"(
+                     dk::smem_u32(bar))
+                 : "memory");
+}
+__device__ __forceinline__ void tc_fence_after() { asm volatile("tcgen05.fence::after_thread_sync;" ::: "memory"); }
+__device__ __forceinline__ void tc_fence_before() { asm volatile("tcgen05.fence::before_thread_sync;" ::: "memory"); }
+
+__device__ __forceinline__ void tmem_ld32(uint32_t addr, uint32_t (&v)[32])
+{
+    asm volatile(
+        "tcgen05.ld.sync.aligned.32x32b.x32.b32 {%0,%1,%2,%3,%4,%5,%6,%7,%8,%9,%10,%11,%12,%13,%14,%15,"
+        "%16,%17,%18,%19,%20,%21,%22,%23,%24,%25,%26,%27,%28,%29,%30,%31}, [%32];"
+        : "=r"(v[0]), "=r"(v[1]), "=r"(v[2]), "=r"(v[3]), "=r"(v[4]), "=r"(v[5]), "=r"(v[6]), "=r"(v[7]),
+          "=r"(v[8]), "=r"(v[9]), "=r"(v[10]), "=r"(v[11]), "=r"(v[12]), "=r"(v[13]), "=r"(v[14]), "=r"(v[15]),
+          "=r"(v[16]), "=r"(v[17]), "=r"(v[18]), "=r"(v[19]), "=r"(v[20]), "=r"(v[21]), "=r"(v[22]),
+          "=r"(v[23]), "=r"(v[24]), "=r"(v[25]), "=r"(v[26]), "=r"(v[27]), "=r"(v[28]), "=r"(v[29]),
+          "=r"(v[30]), "=r"(v[31])
+        : "r"(addr));
+    asm volatile("tcgen05.wait::ld.sync.aligned;" ::: "memory");
+}
+
+__device__ __forceinline__ void tma_load_5d(void* dst, const CUtensorMap* map, int c0, int c1, int c2, int c3,
+                                            int c4, uint64_t* bar)
+{
+    asm volatile(
+        "cp.async.bulk.tensor.5d.shared::cluster.global.tile.mbarrier::complete_tx::bytes"
+        " [%0], [%1, {%2, %3, %4, %5, %6}], [%7];" ::"r"(dk::smem_u32(dst)),
+        "l"(reinterpret_cast<uint64_t>(map)), "r"(c0), "r"(c1), "r"(c2), "r"(c3), "r"(c4),
+        "r"(dk::smem_u32(bar))
+        : "memory");
+}
+
+// Sorted (ascending) per-thread key list, fully unrolled insertion.
+__device__ __forceinline__ void list_insert(unsigned long long (&L)[LIST], unsigned long long key)
+{
+#pragma unroll
+    for (int i = LIST - 1; i > 0; i--) {
+        const unsigned long long a = L[i - 1], b = L[i];
+        L[i] = key < a ? a : (key < b ? key : b);
+    }
+    L[0] = key < L[0] ? key : L[0];
+}
+
+template <int M, int Q, int NBUF, bool GRID>
+__global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__ CUtensorMap tmap, const TcArgs a)
+{
+    static_assert(Q * NBUF * NT <= 512, "TMEM has 512 columns");
+    constexpr int MXP = (M + 1) / 2;   // voxel pairs along x (K = 16 = 2 voxels x 8 channels)
+    extern __shared__ __align__(1024) unsigned char smem[];
+    __shared__ uint64_t bars[2 * 2 + 2 * WSTAGES + 2 * NBUF];
+    __shared__ uint32_t tmem_base_s;
+    uint64_t* rec_full = bars;
+    uint64_t* rec_empty = bars + 2;
+    uint64_t* w_full = bars + 4;
+    uint64_t* w_empty = w_full + WSTAGES;
+    uint64_t* tm_full = w_empty + WSTAGES;
+    uint64_t* tm_empty = tm_full + NBUF;
+
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    const int block = blockIdx.x / a.G, region = blockIdx.x % a.G;
+    const int tile_begin = region * a.tiles_per_region;
+    const int tile_end = min(a.ntiles, tile_begin + a.tiles_per_region);
+    const int n_tiles = tile_end - tile_begin;
+    unsigned char* rec_smem = smem;
+    unsigned char* w_smem = smem + a.n_rec_stages * a.rec_stage_bytes;
+
+    if (threadIdx.x == 0) {
+        for (int i = 0; i < 2; i++) {
+            dk::mbar_init(&rec_full[i], 1);
+            dk::mbar_init(&rec_empty[i], 1);
+        }
+        for (int i = 0; i < WSTAGES; i++) {
+            dk::mbar_init(&w_full[i], 1);
+            dk::mbar_init(&w_empty[i], 1);
+        }
+        for (int i = 0; i < NBUF; i++) {
+            dk::mbar_init(&tm_full[i], 1);
+            dk::mbar_init(&tm_empty[i], NEPI);
+        }
+        dk::fence_mbar_init();
+    }
+    if (warp == 1) {
+        asm volatile("tcgen05.alloc.cta_group::1.sync.aligned.shared::cta.b32 [%0], 512;" ::"r"(
+            dk::smem_u32(&tmem_base_s)));
+        asm volatile("tcgen05.relinquish_alloc_permit.cta_group::1.sync.aligned;");
+    }
+    tc_fence_before();
+    __syncthreads();
+    tc_fence_after();
+    const uint32_t tmem = tmem_base_s;
+
+    if (n_tiles > 0) {
+        if (warp == 0) {
+            // ------------------------------------------------ TMA producer
+            if (lane == 0) {
+                dk::prefetch_tmap(&tmap);
+                const unsigned char* wsrc = a.W + static_cast<size_t>(block) * a.nsteps * WCHUNK;
+                int wi = 0;
+                for (int ti = 0; ti < n_tiles; ti++) {
+                    const int tile = tile_begin + ti;
+                    const int rs = ti % a.n_rec_stages, ruse = ti / a.n_rec_stages;
+                    if (ruse > 0) dk::mbar_wait(&rec_empty[rs], (ruse - 1) & 1);
+                    const int tx = tile % a.ntx, ty = (tile / a.ntx) % a.nty, tz = tile / (a.ntx * a.nty);
+                    unsigned char* rdst = rec_smem + static_cast<size_t>(rs) * a.rec_stage_bytes;
+                    dk::mbar_arrive_expect_tx(&rec_full[rs], a.G_ch * a.box_bytes);
+                    for (int g = 0; g < a.G_ch; g++)
+                        tma_load_5d(rdst + static_cast<size_t>(g) * a.box_bytes, &tmap, 0, tx * NT, ty * Q, tz, g,
+                                    &rec_full[rs]);
+                    for (int s = 0; s < a.nsteps; s++, wi++) {
+                        const int ws = wi % WSTAGES, wuse = wi / WSTAGES;
+                        if (wuse > 0) dk::mbar_wait(&w_empty[ws], (wuse - 1) & 1);
+                        dk::mbar_arrive_expect_tx(&w_full[ws], WCHUNK);
+                        dk::bulk_load(w_smem + static_cast<size_t>(ws) * WCHUNK, wsrc + static_cast<size_t>(s) * WCHUNK,
+                                      WCHUNK, &w_full[ws]);
+                    }
+                }
+            }
+        } else if (warp == 1) {
+            // ------------------------------------------------ MMA issuer (one thread)
+            if (lane == 0) {
+                constexpr uint32_t idesc = umma_idesc(ROT, NT);
+                const uint32_t rec0 = dk::smem_u32(rec_smem), w0 = dk::smem_u32(w_smem);
+                int wi = 0;
+                for (int ti = 0; ti < n_tiles; ti++) {
+                    const int rs = ti % a.n_rec_stages, ruse = ti / a.n_rec_stages;
+                    const int buf = ti % NBUF, buse = ti / NBUF;
+                    dk::mbar_wait(&rec_full[rs], ruse & 1);
+                    if (buse > 0) dk::mbar_wait(&tm_empty[buf], (buse - 1) & 1);
+                    tc_fence_after();
+                    const uint32_t rbase = rec0 + rs * a.rec_stage_bytes;
+                    for (int s = 0; s < a.nsteps; s++, wi++) {
+                        const int ws = wi % WSTAGES, wuse = wi / WSTAGES;
+                        dk::mbar_wait(&w_full[ws], wuse & 1);
+                        tc_fence_after();
+                        // step s -> (g, pass, vz, vy, vxp)
+                        const int vxp = s % MXP, vy = (s / MXP) % M, vz = (s / (MXP * M)) % M;
+                        const int g = s / (MXP * M * M * 2);
+                        const uint64_t da = umma_desc(w0 + ws * WCHUNK, ROT * 16, 128);
+                        const uint32_t bq =
+                            rbase + g * a.box_bytes + ((vz * a.TYB + vy) * a.TXB + 2 * vxp) * 16;
+#pragma unroll
+                        for (int q = 0; q < Q; q++) {
+                            const uint64_t db = umma_desc(bq + q * a.TXB * 16, 16, 128);
+                            umma_bf16(tmem + (buf * Q + q) * NT, da, db, idesc, s > 0 ? 1u : 0u);
+                        }
+                        umma_commit(&w_empty[ws]);
+                    }
+                    umma_commit(&tm_full[buf]);
+                    umma_commit(&rec_empty[rs]);
+                }
+            }
+        } else {
+            // ------------------------------------------------ epilogue warps
+            const int quarter = warp & 3;
+            const int half = (warp - 2) >> 2;
+            const int r = quarter * 32 + lane;                  // rotation within the block (TMEM lane)
+            const int slot = block * ROT + r;
+            const bool rot_ok = slot < a.n_slots;
+            unsigned long long lst[LIST];
+#pragma unroll
+            for (int i = 0; i < LIST; i++) lst[i] = KEY_MAX;
+            float th = __int_as_float(0x7f800000);
+            for (int ti = 0; ti < n_tiles; ti++) {
+                const int tile = tile_begin + ti;
+                const int buf = ti % NBUF, buse = ti / NBUF;
+                dk::mbar_wait(&tm_full[buf], buse & 1);
+                tc_fence_after();
+                const int tx = tile % a.ntx, ty = (tile / a.ntx) % a.nty, tz = tile / (a.ntx * a.nty);
+                for (int q = half; q < Q; q += 2) {
+                    const int y = ty * Q + q, z = tz;
+                    const bool row_ok = rot_ok && y < a.ny && z < a.nz;
+                    const int x0 = tx * NT;
+                    const uint32_t tbase = static_cast<uint32_t>((z * a.ny + y) * a.nx + x0);
+#pragma unroll 1
+                    for (int c0 = 0; c0 < NT; c0 += 32) {
+                        uint32_t v[32];
+                        tmem_ld32(tmem + (static_cast<uint32_t>(quarter * 32) << 16) + (buf * Q + q) * NT + c0, v);
+                        if (!row_ok) continue;
+                        if constexpr (GRID) {
+                            float* out = a.grid + static_cast<size_t>(slot) * a.nx * a.ny * a.nz + tbase;
+#pragma unroll
+                            for (int j = 0; j < 32; j++)
+                                if (x0 + c0 + j < a.nx) out[c0 + j] = __uint_as_float(v[j]);
+                        } else {
+#pragma unroll
+                            for (int j = 0; j < 32; j++) {
+                                const float sv = __uint_as_float(v[j]);
+                                if (sv <= th && x0 + c0 + j < a.nx) {
+                                    const unsigned long long key = dk::make_key(sv, tbase + c0 + j);
+                                    if (key < lst[LIST - 1]) {
+                                        list_insert(lst, key);
+                                        th = dk::key_score_bound(static_cast<uint32_t>(lst[LIST - 1] >> 32));
+                                    }
+                                }
+                            }
+                        }
+                    }
+                }
+                tc_fence_before();
+                __syncwarp();
+                if (lane == 0) dk::mbar_arrive(&tm_empty[buf]);
+            }
+            if constexpr (!GRID) {
+                if (rot_ok) {
+                    // bound: k list entries pairwise farther than 2*rho apart
+                    unsigned long long Tw = KEY_MAX;
+                    uint32_t chosen[dk::RB * 4];
+                    int nc = 0;
+                    for (int i = 0; i < LIST && nc < a.k; i++) {
+                        if (lst[i] == KEY_MAX) break;
+                        const uint32_t t = static_cast<uint32_t>(lst[i] & 0xffffffffu);
+                        bool far = true;
+                        for (int c = 0; c < nc; c++)
+                            far = far && dk::cheb_cyc(t, chosen[c], a.nx, a.ny, a.nz) > 2 * a.rho;
+                        if (far) {
+                            chosen[nc++] = t;
+                            if (nc == a.k) Tw = lst[i];
+                        }
+                    }
+                    const unsigned long long old = atomicMin(&a.T[slot], Tw);
+                    const unsigned long long Tn = old < Tw ? old : Tw;
+                    atomicMin(&a.mu[slot], lst[LIST - 1]);
+                    for (int i = 0; i < LIST; i++) {
+                        if (lst[i] == KEY_MAX || lst[i] > Tn) break;
+                        const unsigned pos = atomicAdd(&a.cnt[slot], 1u);
+                        if (pos < static_cast<unsigned>(a.cap)) a.cand[static_cast<size_t>(slot) * a.cap + pos] = lst[i];
+                    }
+                }
+            }
+        }
+    }
+    tc_fence_before();
+    __syncthreads();
+    if (warp == 1) asm volatile("tcgen05.dealloc.cta_group::1.sync.aligned.b32 %0, 512;" ::"r"(tmem));
+}
+
+// ------------------------------------------------------------------ data preparation
+
+// bf16 split of the padded receptor: Rb[g][Z][Y][X][8] = (hi_0..3, lo_0..3) of channels 4g..4g+3
+__global__ void k_pack_receptor_tc(const float* __restrict__ R, uint16_t* __restrict__ Rb, int nx, int ny, int nz,
+                                   int Xp, int Yp, int Zp, int P, int G_ch)
+{
+    const size_t total = static_cast<size_t>(G_ch) * Zp * Yp * Xp;
+    for (size_t i = blockIdx.x * static_cast<size_t>(blockDim.x) + threadIdx.x; i < total;
+         i += static_cast<size_t>(gridDim.x) * blockDim.x) {
+        const int X = static_cast<int>(i % Xp);
+        size_t rr = i / Xp;
+        const int Y = static_cast<int>(rr % Yp);
+        rr /= Yp;
+        const int Z = static_cast<int>(rr % Zp);
+        const int g = static_cast<int>(rr / Zp);
+        uint16_t out[8];
+#pragma unroll
+        for (int c = 0; c < 4; c++) {
+            const int p = 4 * g + c;
+            float f = 0.f;
+            if (p < P) f = R[((static_cast<size_t>(p) * nz + Z % nz) * ny + Y % ny) * nx + X % nx];
+            const __nv_bfloat16 hi = __float2bfloat16_rn(f);
+            const __nv_bfloat16 lo = __float2bfloat16_rn(f - __bfloat162float(hi));
+            out[c] = __bfloat16_as_ushort(hi);
+            out[4 + c] = __bfloat16_as_ushort(lo);
+        }
+        uint4 pk;
+        pk.x = out[0] | (static_cast<uint32_t>(out[1]) << 16);
+        pk.y = out[2] | (static_cast<uint32_t>(out[3]) << 16);
+        pk.z = out[4] | (static_cast<uint32_t>(out[5]) << 16);
+        pk.w = out[6] | (static_cast<uint32_t>(out[7]) << 16);
+        reinterpret_cast<uint4*>(Rb)[i] = pk;
+    }
+}
+
+// Folded weights Lw [batch][P][m^3][RB] (k_voxelize output) -> A operand [block][step][chunk][rot][8].
+__global__ void k_pack_weights_tc(const float* __restrict__ Lw, unsigned char* __restrict__ W, int n_slots, int P,
+                                  int G_ch, int m, int nsteps)
+{
+    const int MXP = (m + 1) / 2, m3 = m * m * m;
+    const long long n_blocks = (n_slots + ROT - 1) / ROT;
+    const long long total = n_blocks * nsteps * 2 * ROT;   // one thread per (block, step, chunk, rot) 16-B row
+    for (long long i = blockIdx.x * static_cast<long long>(blockDim.x) + threadIdx.x; i < total;
+         i += static_cast<long long>(gridDim.x) * blockDim.x) {
+        const int r = static_cast<int>(i % ROT);
+        const int c = static_cast<int>((i / ROT) % 2);
+        const int s = static_cast<int>((i / (2 * ROT)) % nsteps);
+        const long long blk = i / (2LL * ROT * nsteps);
+        const int vxp = s % MXP, vy = (s / MXP) % m, vz = (s / (MXP * m)) % m;
+        const int pass = (s / (MXP * m * m)) % 2, g = s / (MXP * m * m * 2);
+        const int vx = 2 * vxp + c;
+        const long long slot = blk * ROT + r;
+        uint16_t out[8] = {0, 0, 0, 0, 0, 0, 0, 0};
+        if (slot < n_slots && vx < m) {
+            const int v = (vz * m + vy) * m + vx;
+#pragma unroll
+            for (int cc = 0; cc < 4; cc++) {
+                const int p = 4 * g + cc;
+                if (p >= P) continue;
+                const float f = Lw[((static_cast<size_t>(slot / dk::RB) * P + p) * m3 + v) * dk::RB + slot % dk::RB];
+                const __nv_bfloat16 hi = __float2bfloat16_rn(f);
+                const __nv_bfloat16 lo = __float2bfloat16_rn(f - __bfloat162float(hi));
+                if (pass == 0) {
+                    out[cc] = __bfloat16_as_ushort(hi);
+                    out[4 + cc] = __bfloat16_as_ushort(hi);
+                } else {
+                    out[cc] = __bfloat16_as_ushort(lo);
+                }
+            }
+        }
+        uint4 pk;
+        pk.x = out[0] | (static_cast<uint32_t>(out[1]) << 16);
+        pk.y = out[2] | (static_cast<uint32_t>(out[3]) << 16);
+        pk.z = out[4] | (static_cast<uint32_t>(out[5]) << 16);
+        pk.w = out[6] | (static_cast<uint32_t>(out[7]) << 16);
+        reinterpret_cast<uint4*>(W)[i] = pk;
+    }
+}
+
+}  // namespace tc
