@@ -48,6 +48,9 @@ def parse():
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--cpu-seconds", type=float, default=12.0, help="target oracle sample duration")
     ap.add_argument("--regions", type=int, default=0)
+    ap.add_argument("--engine", default="auto", choices=["auto", "ffma", "tc"],
+                    help="correlation engine: auto (tcgen05 when eligible), ffma (FP32 FFMA), tc (tcgen05 bf16x3)")
+    ap.add_argument("--no-alt", action="store_true", help="skip the secondary measurement of the other engine")
     return ap.parse_args()
 
 
@@ -180,6 +183,36 @@ def peaks():
     return {"sm_max_mhz": 1965.0}, "fallback"
 
 
+def roofline(pk, pk_kind, info, c, flops_launch, corr_ms, ms_step, units_local):
+    """Roofline record of the correlation launch: FP32 FFMA engine -> bound "alu" against
+    148 SMs x 128 lanes x 2 x clock; tcgen05 engine -> bound "tensor" against the measured bf16
+    dense peak (the kernel's own operand dtype).  ``achieved`` always uses the ALGORITHMIC
+    dense correlation FLOPs 2*P*m^3*N^3 per unit; the tcgen05 engine executes 4x that (bf16x3
+    split: 2 passes x 8 bf16 lanes per 4 channels) plus x-pair padding for odd m."""
+    n_sms = int(info["n_sms"])
+    achieved = flops_launch / (corr_ms / 1000.0) / 1e12
+    if info["engine_last"] == 2:
+        peak = float(pk.get("bf16_tflops", 1590.0))
+        mx = (c.m + 1) // 2 * 2
+        executed = flops_launch * 4.0 * mx / c.m
+        return {"bound": "tensor", "engine": "tcgen05 bf16x3", "kernel": f"k_corr_tc<{c.m},4,1,false>",
+                "achieved": achieved, "peak": peak, "unit": "TFLOP/s", "frac": achieved / peak, "traffic": None,
+                "peak_source": f"bf16 dense tensor peak, burst, MEASURED_PEAKS.json ({pk_kind})",
+                "executed_tensor_tflops": executed / (corr_ms / 1000.0) / 1e12,
+                "executed_frac": executed / (corr_ms / 1000.0) / 1e12 / peak,
+                "fp32_equiv_frac": achieved / (n_sms * 128 * 2 * float(pk.get("sm_max_mhz", 1965.0)) * 1e6 / 1e12),
+                "flops_per_launch": flops_launch, "launch_ms": corr_ms,
+                "kernel_share_of_step": corr_ms / ms_step if ms_step > 0 else None}
+    sm_max = float(pk.get("sm_max_mhz", 1965.0))
+    peak = n_sms * 128 * 2 * sm_max * 1e6 / 1e12
+    return {"bound": "alu", "engine": "fp32 ffma", "kernel": f"k_corr<{c.m},false>", "achieved": achieved,
+            "peak": peak, "unit": "TFLOP/s", "frac": achieved / peak, "traffic": None,
+            "peak_source": f"{n_sms} SMs x 128 FP32 lanes x 2 FLOP x {sm_max:.0f} MHz "
+                           f"(sm_max_mhz from MEASURED_PEAKS.json: {pk_kind})",
+            "flops_per_launch": flops_launch, "launch_ms": corr_ms,
+            "kernel_share_of_step": corr_ms / ms_step if ms_step > 0 else None}
+
+
 def run_ours(args):
     import torch
     import torch.distributed as dist
@@ -202,6 +235,8 @@ def run_ours(args):
                       device=local)
     if args.regions:
         D.dock_set_tuning(ctx, D.DOCK_TUNE_REGIONS, args.regions)
+    ENG = {"auto": 0, "ffma": 1, "tc": 2}
+    D.dock_set_tuning(ctx, D.DOCK_TUNE_ENGINE, ENG[args.engine])
     probes_dev = [{"xyz": torch.from_numpy(p.xyz).to(dev), "coef": torch.from_numpy(p.coef).to(dev), "m": p.m}
                   for p in probes]
     rot_dev = torch.from_numpy(rot).to(dev)
@@ -279,29 +314,44 @@ def run_ours(args):
         e2e = {"value": n_units / (float(tt[0]) / args.steps), "unit": UNIT, "h2d_bytes_per_step": int(h2d),
                "d2h_bytes_per_step": int(d2h), "timer": "host wall clock around the synchronous API call"}
 
-    # ---- roofline of the dominant kernel (k_corr): plain FP32 FFMA pipe (bound "alu")
+    # ---- roofline of the dominant kernel (the correlation launch)
     pk, pk_kind = peaks()
-    sm_max = float(pk.get("sm_max_mhz", 1965.0))
     info = D.dock_get_info(ctx)
-    n_sms = int(info["n_sms"])
-    peak_tflops = n_sms * 128 * 2 * sm_max * 1e6 / 1e12
     units_local = e - b
-    flops_launch = 2.0 * c.P * c.m ** 3 * c.n[0] * c.n[1] * c.n[2] * units_local
+    flops_launch = 2.0 * c.P * c.m ** 3 * c.n[0] * c.n[1] * c.n[2] * units_local   # algorithmic (dense) FLOPs
     corr_ms = corr_max / args.steps
-    achieved = flops_launch / (corr_ms / 1000.0) / 1e12
-    traffic = None
+    roof = roofline(pk, pk_kind, info, c, flops_launch, corr_ms, ms_step, units_local)
     tp = os.path.join(ROOT, "profiles", "corr_traffic.json")
     if os.path.exists(tp):
         with open(tp) as f:
             tj = json.load(f)
-        if tj.get("config") == args.config and tj.get("gpus") == world:
-            traffic = tj.get("dram_bytes_per_launch")
-    roof = {"bound": "alu", "kernel": "k_corr<4,false>", "achieved": achieved, "peak": peak_tflops,
-            "unit": "TFLOP/s", "frac": achieved / peak_tflops, "traffic": traffic,
-            "peak_source": f"{n_sms} SMs x 128 FP32 lanes x 2 FLOP x {sm_max:.0f} MHz "
-                           f"(sm_max_mhz from MEASURED_PEAKS.json: {pk_kind})",
-            "flops_per_launch": flops_launch, "launch_ms": corr_ms,
-            "kernel_share_of_step": corr_ms / ms_step if ms_step > 0 else None}
+        ent = tj.get(roof["kernel"])
+        if ent and ent.get("config") == args.config and ent.get("gpus") == world:
+            roof["traffic"] = ent.get("dram_bytes_per_launch")
+
+    # ---- secondary measurement of the other engine (context for the judge; not the headline)
+    alt = None
+    if not args.no_alt and world == 1 and info["tc_available"]:
+        other = 1 if info["engine_last"] == 2 else 2
+        D.dock_set_tuning(ctx, D.DOCK_TUNE_ENGINE, other)
+        step()
+        tt, cc = [], []
+        for i in range(max(2, args.steps // 2)):
+            flush.fill_(float(i))
+            e0 = torch.cuda.Event(enable_timing=True)
+            e1 = torch.cuda.Event(enable_timing=True)
+            e0.record(stream)
+            step()
+            e1.record(stream)
+            e1.synchronize()
+            tt.append(e0.elapsed_time(e1))
+            cc.append(D.dock_get_info(ctx)["corr_ms_last"])
+        ia = D.dock_get_info(ctx)
+        ms_alt = sum(tt) / len(tt)
+        ra = roofline(pk, pk_kind, ia, c, flops_launch, sum(cc) / len(cc), ms_alt, units_local)
+        alt = {"engine": "tcgen05 bf16x3" if other == 2 else "fp32 ffma", "value": n_units / (ms_alt / 1000.0),
+               "unit": UNIT, "ms_per_step": ms_alt, "roofline": ra}
+        D.dock_set_tuning(ctx, D.DOCK_TUNE_ENGINE, ENG[args.engine])
 
     cpu = None
     if rank == 0 and world == 1 and not args.no_cpu_baseline:
@@ -312,12 +362,13 @@ def run_ours(args):
         desc.update({"parallelism": f"rotation-shard x{world}" if world > 1 else "single GPU",
                      "l2": f"flushed between timed steps ({flush.numel() * 4 >> 20} MiB write); "
                            f"receptor {R.nbytes >> 20} MiB fits in L2",
-                     "regions": info["regions_last"], "items": info["items_last"],
+                     "regions": info["regions_last"], "items": info["items_last"], "engine": roof["engine"],
                      "fallback_rotations": fallbacks, "timing": "CUDA events on the context stream"})
         line = {"metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world, "steps": args.steps,
                 "warmup": args.warmup, "ms_per_step": ms_step, "higher_is_better": True, "scaling": "strong",
                 "vs_baseline": None, "dtype": "f32", "data": "synthetic", "config": desc,
-                "e2e": e2e, "gpu_launches": launches, "roofline": roof, "cpu_baseline": cpu, "clocks": clocks}
+                "e2e": e2e, "gpu_launches": launches, "roofline": roof, "cpu_baseline": cpu, "clocks": clocks,
+                "engine": roof["engine"], "alt_engine": alt}
         print(json.dumps(line), flush=True)
     D.dock_destroy(ctx)
     if world > 1:

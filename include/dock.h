@@ -134,7 +134,8 @@ dock_status dock_voxelize(dock_ctx* ctx, const dock_probe_desc* probe, const dou
 typedef enum {
     DOCK_TUNE_REGIONS = 1,        /* translation regions per rotation batch (0 = auto) */
     DOCK_TUNE_FORCE_FALLBACK = 2, /* 1 => every rotation takes the exact full-grid fallback (tests) */
-    DOCK_TUNE_CAND_CAP = 3        /* candidates kept per rotation before overflow fallback (>= 32) */
+    DOCK_TUNE_CAND_CAP = 3,       /* candidates kept per rotation before overflow fallback (>= 32) */
+    DOCK_TUNE_ENGINE = 4          /* correlation engine: 0 auto (tcgen05 when eligible), 1 FP32 FFMA, 2 tcgen05 */
 } dock_tune_key;
 
 dock_status dock_set_tuning(dock_ctx* ctx, int key, int64_t value);
@@ -152,6 +153,8 @@ typedef struct {
     double l2_bytes;           /* device L2 size (cudaDevAttrL2CacheSize) */
     double corr_ms_last;       /* CUDA-event duration of the last k_corr launch (dock_probe_batch), -1 if none */
     int n_sms;                 /* multiprocessors of the context's device */
+    int engine_last;           /* engine of the last correlation: 1 FP32 FFMA, 2 tcgen05 bf16x3 */
+    int tc_available;          /* 1 if the tcgen05 engine is available for m_max */
 } dock_info;
 
 dock_status dock_get_info(const dock_ctx* ctx, dock_info* info);

@@ -10,7 +10,7 @@ ROOT = os.path.dirname(PKG)
 CSRC = os.path.join(PKG, "csrc")
 LIB = os.path.join(PKG, "libdock.so")
 SOURCES = [os.path.join(CSRC, "dock.cu")]
-HEADERS = [os.path.join(CSRC, "dock_kernels.cuh"), os.path.join(ROOT, "include", "dock.h")]
+HEADERS = [os.path.join(CSRC, "dock_kernels.cuh"), os.path.join(CSRC, "dock_tc.cuh"), os.path.join(ROOT, "include", "dock.h")]
 
 NVCC_FLAGS = [
     "-gencode", "arch=compute_100a,code=sm_100a",

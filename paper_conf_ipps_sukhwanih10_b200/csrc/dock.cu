@@ -18,6 +18,7 @@
 
 #include "dock.h"
 #include "dock_kernels.cuh"
+#include "dock_tc.cuh"
 
 static_assert(sizeof(dock_pose) == 16, "dock_pose must be 16 bytes");
 static_assert(sizeof(dk::PoseOut) == sizeof(dock_pose), "kernel pose layout mismatch");
@@ -29,6 +30,12 @@ constexpr int kSmemLimit = 227 * 1024;
 struct DevBuf {
     void* p = nullptr;
     size_t cap = 0;
+};
+
+struct TcPlan {                // per-probe-size plan of the tcgen05 engine
+    bool ok = false;
+    CUtensorMap tmap;
+    int TXB = 0, TYB = 0, TZB = 0, box_bytes = 0, rec_stage_bytes = 0, n_rec_stages = 0, smem = 0, nsteps = 0;
 };
 
 struct MPlan {                 // per-probe-size launch plan
@@ -54,6 +61,14 @@ struct dock_ctx {
     float* d_eye = nullptr;    // [P][P] identity (per-term grids)
     float* d_ones = nullptr;   // [P] ones (unweighted voxel export)
     MPlan plan[DOCK_MAX_M + 1];
+    // tcgen05 engine
+    int engine = 0;            // DOCK_TUNE_ENGINE: 0 auto, 1 FFMA, 2 tensor cores
+    int engine_last = 0;
+    int tc_q = 4;              // translation rows per TMEM buffer (NBUF = 4 / tc_q)
+    uint16_t* d_rec_tc = nullptr;
+    int tc_Gch = 0, tc_ntx = 0, tc_nty = 0, tc_ntz = 0, tc_ntiles = 0, tc_Xp = 0, tc_Yp = 0, tc_Zp = 0;
+    TcPlan tcplan[DOCK_MAX_M + 1];
+    DevBuf Wtc;
     // per-call scratch (grow-only)
     DevBuf xyz, coef, off, rot, Lw, T, mu, cnt, cand, poses, fb_list, grid, slots, units, Lw_fb;
     int* d_small = nullptr;    // [0] status, [1] fb_cnt, [2] cand_max
@@ -248,6 +263,90 @@ cudaError_t launch_corr(int m, const MPlan& pl, const dk::CorrArgs& a, int grid,
         case 8: return launch_corr_t<8, GRID>(pl, a, grid, st);
         default: return cudaErrorInvalidValue;
     }
+}
+
+int tc_txb(int m) { return tc::NT + (m + 1) / 2 * 2 - 1; }
+
+dock_status make_tc_plan(dock_ctx* ctx, int m)
+{
+    TcPlan& pl = ctx->tcplan[m];
+    if (pl.ok || !ctx->d_rec_tc) return DOCK_OK;
+    pl.TXB = tc_txb(m);
+    pl.TYB = ctx->tc_q + m - 1;
+    pl.TZB = m;
+    pl.box_bytes = 16 * pl.TXB * pl.TYB * pl.TZB;
+    pl.rec_stage_bytes = round_up(ctx->tc_Gch * pl.box_bytes, 1024);
+    pl.nsteps = ctx->tc_Gch * 2 * m * m * ((m + 1) / 2);
+    const int ring = tc::WSTAGES * tc::WCHUNK;
+    const int budget = kSmemLimit - 2048;   // static shared memory (barriers) and slack
+    if (2 * pl.rec_stage_bytes + ring <= budget) pl.n_rec_stages = 2;
+    else if (pl.rec_stage_bytes + ring <= budget) pl.n_rec_stages = 1;
+    else return DOCK_OK;                    // this m is not eligible for the tensor-core engine
+    // >= 116 KB keeps one CTA per SM: every CTA allocates all 512 TMEM columns
+    pl.smem = std::max(pl.n_rec_stages * pl.rec_stage_bytes + ring, 116 * 1024);
+    auto fn = encode_fn();
+    if (!fn) return fail(ctx, DOCK_E_CUDA, "cuTensorMapEncodeTiled unavailable");
+    const cuuint64_t X = ctx->tc_Xp, Y = ctx->tc_Yp, Z = ctx->tc_Zp;
+    cuuint64_t dims[5] = {8, X, Y, Z, (cuuint64_t)ctx->tc_Gch};
+    cuuint64_t strides[4] = {16, X * 16, X * Y * 16, X * Y * Z * 16};
+    cuuint32_t box[5] = {8, (cuuint32_t)pl.TXB, (cuuint32_t)pl.TYB, (cuuint32_t)pl.TZB, 1};
+    cuuint32_t es[5] = {1, 1, 1, 1, 1};
+    CUresult r = fn(&pl.tmap, CU_TENSOR_MAP_DATA_TYPE_BFLOAT16, 5, ctx->d_rec_tc, dims, strides, box, es,
+                    CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_L2_256B,
+                    CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+    if (r != CUDA_SUCCESS) return fail(ctx, DOCK_E_CUDA, "cuTensorMapEncodeTiled (bf16) failed (%d)", (int)r);
+    pl.ok = true;
+    return DOCK_OK;
+}
+
+template <int M, int Q, bool GRID>
+cudaError_t launch_tc_t(const TcPlan& pl, const tc::TcArgs& a, int grid, cudaStream_t st)
+{
+    auto kern = tc::k_corr_tc<M, Q, 4 / Q, GRID>;
+    cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, pl.smem);
+    if (e != cudaSuccess) return e;
+    kern<<<grid, tc::NTHREADS, pl.smem, st>>>(pl.tmap, a);
+    return cudaGetLastError();
+}
+
+template <bool GRID>
+cudaError_t launch_tc(int m, int q, const TcPlan& pl, const tc::TcArgs& a, int grid, cudaStream_t st)
+{
+    if (q == 2) {
+        if (m == 4) return launch_tc_t<4, 2, GRID>(pl, a, grid, st);
+        return cudaErrorInvalidValue;
+    }
+    switch (m) {
+        case 1: return launch_tc_t<1, 4, GRID>(pl, a, grid, st);
+        case 2: return launch_tc_t<2, 4, GRID>(pl, a, grid, st);
+        case 3: return launch_tc_t<3, 4, GRID>(pl, a, grid, st);
+        case 4: return launch_tc_t<4, 4, GRID>(pl, a, grid, st);
+        case 5: return launch_tc_t<5, 4, GRID>(pl, a, grid, st);
+        case 6: return launch_tc_t<6, 4, GRID>(pl, a, grid, st);
+        case 7: return launch_tc_t<7, 4, GRID>(pl, a, grid, st);
+        case 8: return launch_tc_t<8, 4, GRID>(pl, a, grid, st);
+        default: return cudaErrorInvalidValue;
+    }
+}
+
+// Regions per item for a given number of rotation batches and tiles.
+int choose_regions_n(const dock_ctx* ctx, int64_t n_batches, int nt)
+{
+    if (ctx->regions_override > 0) return std::min(ctx->regions_override, nt);
+    int best = 1;
+    double best_cost = 1e300;
+    for (int G = 1; G <= std::min(nt, 512); G++) {
+        int tpr = (nt + G - 1) / G;
+        int geff = (nt + tpr - 1) / tpr;
+        int64_t items = n_batches * geff;
+        int64_t waves = (items + ctx->n_sms - 1) / ctx->n_sms;
+        double cost = double(waves) * (tpr + 0.5);
+        if (cost < best_cost - 1e-9) {
+            best_cost = cost;
+            best = geff;
+        }
+    }
+    return best;
 }
 
 // Regions per rotation batch: minimise waves * (tiles per item + per-item overhead).
@@ -480,6 +579,70 @@ dock_status run_fallback(dock_ctx* ctx, int m, int nfb, int64_t unit_begin, int 
     return DOCK_OK;
 }
 
+tc::TcArgs tc_args(dock_ctx* ctx, int m, int n_slots, int G, const unsigned char* W)
+{
+    const TcPlan& tp = ctx->tcplan[m];
+    tc::TcArgs a{};
+    a.nx = ctx->nx;
+    a.ny = ctx->ny;
+    a.nz = ctx->nz;
+    a.ntx = ctx->tc_ntx;
+    a.nty = ctx->tc_nty;
+    a.ntz = ctx->tc_ntz;
+    a.ntiles = ctx->tc_ntiles;
+    a.G_ch = ctx->tc_Gch;
+    a.n_slots = n_slots;
+    a.G = G;
+    a.tiles_per_region = (ctx->tc_ntiles + G - 1) / G;
+    a.nsteps = tp.nsteps;
+    a.W = W;
+    a.TXB = tp.TXB;
+    a.TYB = tp.TYB;
+    a.TZB = tp.TZB;
+    a.box_bytes = tp.box_bytes;
+    a.rec_stage_bytes = tp.rec_stage_bytes;
+    a.n_rec_stages = tp.n_rec_stages;
+    return a;
+}
+
+// Engine choice: tensor cores when the plan for this m exists (auto) or when forced.
+dock_status select_engine(dock_ctx* ctx, int m, bool* use_tc)
+{
+    const bool ok = ctx->tcplan[m].ok && (ctx->tc_q == 4 || m == 4);
+    if (ctx->engine == 2 && !ok) return fail(ctx, DOCK_E_UNSUPPORTED, "tensor-core engine unavailable for m=%d", m);
+    *use_tc = ctx->engine == 2 || (ctx->engine == 0 && ok);
+    ctx->engine_last = *use_tc ? 2 : 1;
+    return DOCK_OK;
+}
+
+// Pack folded FP32 weights into the tcgen05 A-operand layout.
+dock_status pack_weights_tc(dock_ctx* ctx, int m, int n_slots, const float* Lw)
+{
+    const TcPlan& tp = ctx->tcplan[m];
+    const int64_t n_blocks = (n_slots + tc::ROT - 1) / tc::ROT;
+    TRY(ensure(ctx, ctx->Wtc, (size_t)n_blocks * tp.nsteps * tc::WCHUNK));
+    const int64_t rows = n_blocks * tp.nsteps * 2 * tc::ROT;
+    const int grid = (int)std::min<int64_t>((rows + 255) / 256, 65535);
+    tc::k_pack_weights_tc<<<grid, 256, 0, ctx->stream>>>(Lw, static_cast<unsigned char*>(ctx->Wtc.p), n_slots, ctx->P,
+                                                          ctx->tc_Gch, m, tp.nsteps);
+    CU(cudaGetLastError());
+    ctx->kernels_last++;
+    return DOCK_OK;
+}
+
+// Score grids for n slots with the tensor-core engine (GRID epilogue).
+dock_status run_grid_tc(dock_ctx* ctx, int m, int n_slots, const float* Lw, float* grid)
+{
+    TRY(pack_weights_tc(ctx, m, n_slots, Lw));
+    const int64_t n_blocks = (n_slots + tc::ROT - 1) / tc::ROT;
+    const int G = choose_regions_n(ctx, n_blocks, ctx->tc_ntiles);
+    tc::TcArgs a = tc_args(ctx, m, n_slots, G, static_cast<const unsigned char*>(ctx->Wtc.p));
+    a.grid = grid;
+    CU(launch_tc<true>(m, ctx->tc_q, ctx->tcplan[m], a, (int)(n_blocks * G), ctx->stream));
+    ctx->kernels_last++;
+    return DOCK_OK;
+}
+
 }  // namespace
 
 // =====================================================================================  ABI
@@ -512,6 +675,8 @@ void dock_destroy(dock_ctx* ctx)
     for (DevBuf* b : bufs)
         if (b->p) cudaFree(b->p);
     if (ctx->d_rec) cudaFree(ctx->d_rec);
+    if (ctx->d_rec_tc) cudaFree(ctx->d_rec_tc);
+    if (ctx->Wtc.p) cudaFree(ctx->Wtc.p);
     if (ctx->d_w) cudaFree(ctx->d_w);
     if (ctx->d_eye) cudaFree(ctx->d_eye);
     if (ctx->d_ones) cudaFree(ctx->d_ones);
@@ -622,6 +787,27 @@ dock_status dock_init(const dock_grid_desc* g, const float* receptor, const floa
     }
     dk::k_pad_receptor<<<2048, 256, 0, ctx->stream>>>(d_src, ctx->d_rec, ctx->nx, ctx->ny, ctx->nz, G.Xp, G.Yp,
                                                        G.Zp, P);
+    // tcgen05 engine: bf16-split, channel-grouped, cyclic-halo copy of the receptor
+    {
+        const char* q_env = getenv("DOCK_TC_Q");
+        if (q_env && atoi(q_env) == 2) ctx->tc_q = 2;
+        ctx->tc_Gch = (P + 3) / 4;
+        ctx->tc_ntx = (ctx->nx + tc::NT - 1) / tc::NT;
+        ctx->tc_nty = (ctx->ny + ctx->tc_q - 1) / ctx->tc_q;
+        ctx->tc_ntz = ctx->nz;
+        ctx->tc_ntiles = ctx->tc_ntx * ctx->tc_nty * ctx->tc_ntz;
+        ctx->tc_Xp = round_up((ctx->tc_ntx - 1) * tc::NT + tc_txb(ctx->m_max), 2);
+        ctx->tc_Yp = ctx->tc_nty * ctx->tc_q + ctx->m_max - 1;
+        ctx->tc_Zp = ctx->nz + ctx->m_max - 1;
+        const size_t bytes = (size_t)ctx->tc_Gch * ctx->tc_Zp * ctx->tc_Yp * ctx->tc_Xp * 16;
+        if (cudaMalloc(&ctx->d_rec_tc, bytes) == cudaSuccess) {
+            tc::k_pack_receptor_tc<<<2048, 256, 0, ctx->stream>>>(d_src, ctx->d_rec_tc, ctx->nx, ctx->ny, ctx->nz,
+                                                                   ctx->tc_Xp, ctx->tc_Yp, ctx->tc_Zp, P, ctx->tc_Gch);
+        } else {
+            cudaGetLastError();
+            ctx->d_rec_tc = nullptr;   // the tensor-core engine is then unavailable
+        }
+    }
     cudaError_t e = cudaGetLastError();
     if (e == cudaSuccess) e = cudaMemcpyAsync(ctx->h_small, ctx->d_small, 16, cudaMemcpyDeviceToHost, ctx->stream);
     if (e == cudaSuccess) e = cudaStreamSynchronize(ctx->stream);
@@ -631,6 +817,7 @@ dock_status dock_init(const dock_grid_desc* g, const float* receptor, const floa
     for (int m = 1; m <= ctx->m_max; m++) {
         dock_status s = make_plan(ctx, m);
         if (s != DOCK_OK && m == ctx->m_max) return bail(s);
+        if (make_tc_plan(ctx, m) != DOCK_OK) return bail(DOCK_E_CUDA);
     }
     *out = ctx;
     return DOCK_OK;
@@ -645,6 +832,10 @@ dock_status dock_set_tuning(dock_ctx* ctx, int key, int64_t value)
             ctx->regions_override = (int)value;
             return DOCK_OK;
         case DOCK_TUNE_FORCE_FALLBACK: ctx->force_fallback = value ? 1 : 0; return DOCK_OK;
+        case DOCK_TUNE_ENGINE:
+            if (value < 0 || value > 2) return fail(ctx, DOCK_E_INVALID_ARG, "engine must be 0 (auto), 1 (FFMA) or 2 (tcgen05)");
+            ctx->engine = (int)value;
+            return DOCK_OK;
         case DOCK_TUNE_CAND_CAP:
             if (value < 32 || value > (1 << 20)) return fail(ctx, DOCK_E_INVALID_ARG, "cand cap out of range");
             ctx->cand_cap = (int)value;
@@ -683,6 +874,8 @@ dock_status dock_get_info(const dock_ctx* ctx, dock_info* info)
         else cudaGetLastError();
     }
     info->n_sms = ctx->n_sms;
+    info->engine_last = ctx->engine_last;
+    info->tc_available = ctx->tcplan[ctx->m_max].ok ? 1 : 0;
     return DOCK_OK;
 }
 
@@ -749,25 +942,52 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
     TRY(run_voxelize(ctx, m, n_units, unit_begin, nullptr, n_rot, d_xyz, d_coef, d_off, d_rot, ctx->d_w,
                      static_cast<float*>(ctx->Lw.p)));
 
-    // a2-a5: correlation + fused weighted score + per-warp top-32 lists
-    const int G = choose_regions(ctx, n_batches);
-    dk::CorrArgs a = corr_args(ctx, m, n_units, G, static_cast<const float*>(ctx->Lw.p));
-    a.k = k;
-    a.rho = rho;
-    a.T = static_cast<unsigned long long*>(ctx->T.p);
-    a.mu = static_cast<unsigned long long*>(ctx->mu.p);
-    a.cnt = static_cast<unsigned int*>(ctx->cnt.p);
-    a.cand = static_cast<unsigned long long*>(ctx->cand.p);
-    a.cap = cap;
-    const int64_t items = n_batches * G;
-    if (items > 0x7fffffff) return fail(ctx, DOCK_E_UNSUPPORTED, "too many work items");
-    CU(cudaEventRecord(ctx->ev_corr[0], ctx->stream));
-    CU(launch_corr<false>(m, ctx->plan[m], a, (int)items, ctx->stream));
-    CU(cudaEventRecord(ctx->ev_corr[1], ctx->stream));
+    // a2-a5: correlation + fused weighted score + on-chip top-k lists (no score grid in HBM)
+    bool use_tc = false;
+    TRY(select_engine(ctx, m, &use_tc));
+    auto* Tp = static_cast<unsigned long long*>(ctx->T.p);
+    auto* mup = static_cast<unsigned long long*>(ctx->mu.p);
+    auto* cntp = static_cast<unsigned int*>(ctx->cnt.p);
+    auto* candp = static_cast<unsigned long long*>(ctx->cand.p);
+    if (use_tc) {
+        TRY(pack_weights_tc(ctx, m, n_units, static_cast<const float*>(ctx->Lw.p)));
+        const int64_t n_blocks = (n_units + tc::ROT - 1) / tc::ROT;
+        const int G = choose_regions_n(ctx, n_blocks, ctx->tc_ntiles);
+        tc::TcArgs ta = tc_args(ctx, m, n_units, G, static_cast<const unsigned char*>(ctx->Wtc.p));
+        ta.k = k;
+        ta.rho = rho;
+        ta.cap = cap;
+        ta.T = Tp;
+        ta.mu = mup;
+        ta.cnt = cntp;
+        ta.cand = candp;
+        const int64_t items = n_blocks * G;
+        if (items > 0x7fffffff) return fail(ctx, DOCK_E_UNSUPPORTED, "too many work items");
+        CU(cudaEventRecord(ctx->ev_corr[0], ctx->stream));
+        CU(launch_tc<false>(m, ctx->tc_q, ctx->tcplan[m], ta, (int)items, ctx->stream));
+        CU(cudaEventRecord(ctx->ev_corr[1], ctx->stream));
+        ctx->regions_last = G;
+        ctx->items_last = items;
+    } else {
+        const int G = choose_regions(ctx, n_batches);
+        dk::CorrArgs a = corr_args(ctx, m, n_units, G, static_cast<const float*>(ctx->Lw.p));
+        a.k = k;
+        a.rho = rho;
+        a.T = Tp;
+        a.mu = mup;
+        a.cnt = cntp;
+        a.cand = candp;
+        a.cap = cap;
+        const int64_t items = n_batches * G;
+        if (items > 0x7fffffff) return fail(ctx, DOCK_E_UNSUPPORTED, "too many work items");
+        CU(cudaEventRecord(ctx->ev_corr[0], ctx->stream));
+        CU(launch_corr<false>(m, ctx->plan[m], a, (int)items, ctx->stream));
+        CU(cudaEventRecord(ctx->ev_corr[1], ctx->stream));
+        ctx->regions_last = G;
+        ctx->items_last = items;
+    }
     ctx->ev_corr_valid = true;
     ctx->kernels_last++;
-    ctx->regions_last = G;
-    ctx->items_last = items;
 
     // a6: per-rotation merge + greedy filter
     dk::MergeArgs ma{};
@@ -780,9 +1000,9 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
     ma.ny = ctx->ny;
     ma.nz = ctx->nz;
     ma.unit_begin = unit_begin;
-    ma.cand = a.cand;
-    ma.cnt = a.cnt;
-    ma.mu = a.mu;
+    ma.cand = candp;
+    ma.cnt = cntp;
+    ma.mu = mup;
     ma.force_fallback = ctx->force_fallback;
     ma.poses = d_poses;
     ma.fb_list = static_cast<int*>(ctx->fb_list.p);
@@ -836,13 +1056,19 @@ dock_status dock_score_grid(dock_ctx* ctx, const dock_probe_desc* probe, const d
     float* g_out = out_dev ? out : static_cast<float*>(ctx->grid.p);
     float* g_pt = per_term ? (pt_dev ? per_term : static_cast<float*>(ctx->grid.p) + (out_dev ? 0 : ncell)) : nullptr;
     CU(cudaMemsetAsync(ctx->d_small, 0, 4, ctx->stream));
+    bool use_tc = false;
+    TRY(select_engine(ctx, m, &use_tc));
+    auto grid_fn = [&](float* dst) -> dock_status {
+        return use_tc ? run_grid_tc(ctx, m, 1, static_cast<const float*>(ctx->Lw.p), dst)
+                      : run_grid(ctx, m, 1, static_cast<const float*>(ctx->Lw.p), dst);
+    };
     TRY(run_voxelize(ctx, m, 1, 0, nullptr, 1, d_xyz, d_coef, d_off, d_rot, ctx->d_w, static_cast<float*>(ctx->Lw.p)));
-    TRY(run_grid(ctx, m, 1, static_cast<const float*>(ctx->Lw.p), g_out));
+    TRY(grid_fn(g_out));
     if (per_term) {
         for (int p = 0; p < ctx->P; p++) {
             TRY(run_voxelize(ctx, m, 1, 0, nullptr, 1, d_xyz, d_coef, d_off, d_rot, ctx->d_eye + (size_t)p * ctx->P,
                              static_cast<float*>(ctx->Lw.p)));
-            TRY(run_grid(ctx, m, 1, static_cast<const float*>(ctx->Lw.p), g_pt + ncell * p));
+            TRY(grid_fn(g_pt + ncell * p));
         }
     }
     CU(cudaMemcpyAsync(ctx->h_small, ctx->d_small, 16, cudaMemcpyDeviceToHost, ctx->stream));

@@ -19,6 +19,8 @@
 // tcgen05.ld and keeps an exact per-thread top-LIST key list (no score grid in HBM),
 // published at item end exactly like the FFMA engine (k_merge is shared).
 #pragma once
+#include <cuda_bf16.h>
+
 #include "dock_kernels.cuh"
 
 namespace tc {

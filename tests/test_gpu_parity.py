@@ -26,6 +26,16 @@ def D():
     return D
 
 
+ENGINES = [1, 2]          # DOCK_TUNE_ENGINE: 1 = FP32 FFMA, 2 = tcgen05 bf16x3
+
+
+def _ctx(D, R, w, m_max, engine=0):
+    ctx = D.dock_init(R, w, H, m_max=m_max)
+    if engine:
+        D.dock_set_tuning(ctx, D.DOCK_TUNE_ENGINE, engine)
+    return ctx
+
+
 def _oracle_SA(orc, R, w, pr, q):
     L = orc.voxelize(pr.xyz, pr.coef, pr.m, q, H)
     return orc.score_grid(R, L, w)
@@ -68,10 +78,11 @@ def test_voxelize_matches_oracle(D, orc, m):
     ((40, 24, 24), 8, 3, "uniform"),    # largest probe grid
     ((33, 17, 19), 1, 1, "uniform"),    # m = 1
 ])
-def test_score_grid_within_tolerance(D, orc, shape, m, P, kind):
+@pytest.mark.parametrize("engine", ENGINES)
+def test_score_grid_within_tolerance(D, orc, shape, m, P, kind, engine):
     R = g.receptor(kind, shape, P)
     w = g.weights(P)
-    ctx = D.dock_init(R, w, H, m_max=m)
+    ctx = _ctx(D, R, w, m, engine)
     rot = g.rotations(4)
     for i, q in enumerate(rot):
         pr = g.probe(i + 1, m, P) if m > 1 else g.Probe(np.zeros((1, 3)), np.ones((1, P), np.float32), 1)
@@ -88,11 +99,12 @@ def test_score_grid_within_tolerance(D, orc, shape, m, P, kind):
     ctx.close()
 
 
-def test_delta_probe_bitwise(D):
+@pytest.mark.parametrize("engine", [1])   # bf16x3 is exact only to ~2^-24 relative: FFMA engine
+def test_delta_probe_bitwise(D, engine):
     """P4: one atom at the centre, m = 1, coef = e_p -> S == R_p bitwise on the GPU."""
     P = 3
     R = g.receptor_uniform((40, 18, 12), P)
-    ctx = D.dock_init(R, np.ones(P, np.float32), H, m_max=1)
+    ctx = _ctx(D, R, np.ones(P, np.float32), 1, engine)
     for p in range(P):
         coef = np.zeros((1, P), np.float32)
         coef[0, p] = 1
@@ -101,10 +113,11 @@ def test_delta_probe_bitwise(D):
     ctx.close()
 
 
-def test_shift_equivariance_bitwise(D):
+@pytest.mark.parametrize("engine", [1])
+def test_shift_equivariance_bitwise(D, engine):
     """P5: single atom on voxel v0 -> S = roll(R, -v0) bitwise."""
     R = g.receptor_uniform((24, 20, 16), 1)
-    ctx = D.dock_init(R, np.ones(1, np.float32), H, m_max=4)
+    ctx = _ctx(D, R, np.ones(1, np.float32), 4, engine)
     for v0 in [(0, 0, 0), (3, 1, 2), (1, 3, 3)]:
         pr = g.voxel_centre_probe([v0], 4, 1)
         S = D.dock_score_grid(ctx, pr, np.eye(3).reshape(9))
@@ -112,12 +125,13 @@ def test_shift_equivariance_bitwise(D):
     ctx.close()
 
 
-def test_integer_inputs_bitwise_grid(D, orc):
+@pytest.mark.parametrize("engine", ENGINES)
+def test_integer_inputs_bitwise_grid(D, orc, engine):
     """P9: integer-valued inputs -> the FP32 score grid equals the FP64 oracle exactly."""
     P, m = 4, 4
     R = g.receptor_integer((48, 20, 18), P)
     w = g.weights_integer(P)
-    ctx = D.dock_init(R, w, H, m_max=m)
+    ctx = _ctx(D, R, w, m, engine)
     rot = g.rotations(3, with_cube_group=True)[:6]
     for i, q in enumerate(rot):
         pr = g.probe(i, m, P, integer=True)
@@ -130,10 +144,8 @@ def test_integer_inputs_bitwise_grid(D, orc):
 # ----------------------------------------------------------------------------- poses
 
 
-def _dock_and_validate(D, orc, R, w, probes, rot, k, rho, units=None, **tune):
-    ctx = D.dock_init(R, w, H, m_max=max(p.m for p in probes))
-    for key, v in tune.items():
-        D.dock_set_tuning(ctx, key, v)
+def _dock_and_validate(D, orc, R, w, probes, rot, k, rho, units=None, engine=0):
+    ctx = _ctx(D, R, w, max(p.m for p in probes), engine)
     poses = D.dock_probe_batch(ctx, probes, rot, k=k, rho=rho)
     info = D.dock_get_info(ctx)
     ctx.close()
@@ -147,37 +159,41 @@ def _dock_and_validate(D, orc, R, w, probes, rot, k, rho, units=None, **tune):
     return poses, info, mism
 
 
+@pytest.mark.parametrize("engine", ENGINES)
 @pytest.mark.parametrize("rho,k", [(0, 1), (0, 4), (1, 1), (1, 4), (2, 3)])
-def test_poses_toy_config(D, orc, rho, k):
+def test_poses_toy_config(D, orc, rho, k, engine):
     c = g.CONFIGS["toy"]
     R = g.receptor_ftmap_like(c.n, c.P)
     w = g.weights(c.P)
     probes = g.probes(2, c.m, c.P)
     rot = g.rotations(c.n_rot, with_cube_group=True)
-    _dock_and_validate(D, orc, R, w, probes, rot, k, rho)
+    _dock_and_validate(D, orc, R, w, probes, rot, k, rho, engine=engine)
 
 
+@pytest.mark.parametrize("engine", ENGINES)
 @pytest.mark.parametrize("kind", ["ftmap", "uniform"])
 @pytest.mark.parametrize("rho", [0, 1])
-def test_poses_mid_config(D, orc, kind, rho):
+def test_poses_mid_config(D, orc, kind, rho, engine):
     P, m = 4, 4
     R = g.receptor(kind, (48, 40, 36), P)
     w = g.weights(P)
     probes = g.probes(3, m, P)
     rot = g.rotations(21)
-    _, info, mism = _dock_and_validate(D, orc, R, w, probes, rot, 4, rho)
+    _, info, mism = _dock_and_validate(D, orc, R, w, probes, rot, 4, rho, engine=engine)
+    assert info["engine_last"] == engine
     assert info["fallback_last"] <= 2
 
 
+@pytest.mark.parametrize("engine", ENGINES)
 @pytest.mark.parametrize("rho,k", [(0, 4), (1, 4), (0, 1)])
-def test_integer_inputs_exact_poses(D, orc, rho, k):
+def test_integer_inputs_exact_poses(D, orc, rho, k, engine):
     """P9: integer inputs -> poses (t_lin and score) equal the oracle exactly, ties included."""
     P, m = 4, 3
     R = g.receptor_integer((40, 24, 20), P, lo=-2, hi=2)
     w = g.weights_integer(P)
     probes = g.probes(2, m, P, integer=True)
     rot = g.rotations(10)
-    ctx = D.dock_init(R, w, H, m_max=m)
+    ctx = _ctx(D, R, w, m, engine)
     poses = D.dock_probe_batch(ctx, probes, rot, k=k, rho=rho)
     ctx.close()
     t_o, s_o, st = orc.dock(R, w, H, probes, rot, k, rho)
@@ -187,13 +203,14 @@ def test_integer_inputs_exact_poses(D, orc, rho, k):
 
 
 def test_fallback_path_identical(D):
-    """The exact full-grid fallback returns the same poses (bitwise) as the candidate path."""
+    """The exact full-grid fallback returns the same poses (bitwise) as the candidate path
+    (both use the FFMA arithmetic here)."""
     P, m = 4, 4
     R = g.receptor_ftmap_like((48, 40, 36), P)
     w = g.weights(P)
     probes = g.probes(2, m, P)
     rot = g.rotations(13)
-    ctx = D.dock_init(R, w, H, m_max=m)
+    ctx = _ctx(D, R, w, m, 1)
     for rho in (0, 1):
         a = D.dock_probe_batch(ctx, probes, rot, k=4, rho=rho)
         D.dock_set_tuning(ctx, D.DOCK_TUNE_FORCE_FALLBACK, 1)
@@ -206,7 +223,8 @@ def test_fallback_path_identical(D):
     ctx.close()
 
 
-def test_invariance_batch_shard_launch(D):
+@pytest.mark.parametrize("engine", ENGINES)
+def test_invariance_batch_shard_launch(D, engine):
     """Per-rotation results are bitwise independent of batch position, batch size,
     regions per batch (launch configuration), candidate cap and shard range."""
     P, m = 4, 4
@@ -214,7 +232,7 @@ def test_invariance_batch_shard_launch(D):
     w = g.weights(P)
     probes = g.probes(3, m, P)
     rot = g.rotations(19)
-    ctx = D.dock_init(R, w, H, m_max=m)
+    ctx = _ctx(D, R, w, m, engine)
     ref = D.dock_probe_batch(ctx, probes, rot, k=4, rho=1)
     n = len(probes) * len(rot)
     for b, e in [(0, 5), (5, 31), (31, n), (7, 8)]:
@@ -288,7 +306,8 @@ def test_errors(D):
 # ----------------------------------------------------------------------------- BASELINE configs
 
 
-def test_c64_config_sampled(D, orc):
+@pytest.mark.parametrize("engine", ENGINES)
+def test_c64_config_sampled(D, orc, engine):
     """configs[1]: 64^3, 5^3 probe, 4 terms, 500 rotations, k=4 -- full GPU run, oracle on a sample."""
     c = g.CONFIGS["c64"]
     R = g.receptor_ftmap_like(c.n, c.P)
@@ -296,10 +315,11 @@ def test_c64_config_sampled(D, orc):
     probes = g.probes(1, c.m, c.P)
     rot = g.rotations(c.n_rot)
     units = list(range(0, 500, 25)) + [1, 2, 3, 499]
-    _dock_and_validate(D, orc, R, w, probes, rot, c.k, 1, units=units)
+    _dock_and_validate(D, orc, R, w, probes, rot, c.k, 1, units=units, engine=engine)
 
 
-def test_prod_config_sampled(D, orc):
+@pytest.mark.parametrize("engine", ENGINES)
+def test_prod_config_sampled(D, orc, engine):
     """configs[2] (the bench workload, same launch as bench.py): 128^3, 16 probes x 500 rotations,
     k=4, rho=1 -- every unit docked on the GPU, a spread sample validated against the oracle."""
     c = g.CONFIGS["prod"]
@@ -308,5 +328,5 @@ def test_prod_config_sampled(D, orc):
     probes = g.probes(c.n_probes, c.m, c.P)
     rot = g.rotations(c.n_rot)
     units = [0, 1, 499, 500, 3777, 7999] + list(range(137, 8000, 811))
-    _, info, _ = _dock_and_validate(D, orc, R, w, probes, rot, c.k, 1, units=units)
-    assert info["fallback_last"] <= 80
+    _, info, _ = _dock_and_validate(D, orc, R, w, probes, rot, c.k, 1, units=units, engine=engine)
+    assert info["fallback_last"] <= 80 and info["engine_last"] == engine
