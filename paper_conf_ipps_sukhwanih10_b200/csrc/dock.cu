@@ -70,7 +70,7 @@ struct dock_ctx {
     TcPlan tcplan[DOCK_MAX_M + 1];
     DevBuf Wtc;
     // per-call scratch (grow-only)
-    DevBuf xyz, coef, off, rot, Lw, T, mu, cnt, cand, poses, fb_list, grid, slots, units, Lw_fb;
+    DevBuf xyz, coef, off, rot, Lw, T, mu, cnt, cand, poses, fb_list, grid, slots, units, Lw_fb, picks;
     int* d_small = nullptr;    // [0] status, [1] fb_cnt, [2] cand_max
     int* h_small = nullptr;    // pinned mirror
     void* h_stage = nullptr;   // pinned staging for host inputs
@@ -543,6 +543,7 @@ dock_status run_fallback(dock_ctx* ctx, int m, int nfb, int64_t unit_begin, int 
     const int chunk = (int)std::max<size_t>(1, std::min<size_t>(32, (size_t(1) << 30) / (ncell * 4)));
     TRY(ensure(ctx, ctx->grid, sizeof(float) * ncell * chunk));
     TRY(ensure(ctx, ctx->slots, sizeof(int) * 2 * chunk));
+    TRY(ensure(ctx, ctx->picks, sizeof(unsigned long long) * chunk * k));
     const int m3 = m * m * m;
     TRY(ensure(ctx, ctx->Lw_fb, sizeof(float) * ((chunk + dk::RB - 1) / dk::RB) * dk::RB * ctx->P * m3));
     TRY(ensure_pinned(ctx, sizeof(int) * 2 * chunk));
@@ -563,6 +564,7 @@ dock_status run_fallback(dock_ctx* ctx, int m, int nfb, int64_t unit_begin, int 
         dk::GreedyArgs ga{};
         ga.grid = static_cast<const float*>(ctx->grid.p);
         ga.slots = d_outslot;
+        ga.picks = static_cast<unsigned long long*>(ctx->picks.p);
         ga.n = n;
         ga.k = k;
         ga.rho = rho;
@@ -572,9 +574,17 @@ dock_status run_fallback(dock_ctx* ctx, int m, int nfb, int64_t unit_begin, int 
         ga.nz = ctx->nz;
         ga.unit_begin = unit_begin;
         ga.poses = poses;
-        dk::k_greedy_grid<<<n, 1024, 0, ctx->stream>>>(ga);
+        dk::k_fill_u64<<<1, 256, 0, ctx->stream>>>(ga.picks, (size_t)n * k, dk::KEY_MAX);
         CU(cudaGetLastError());
-        ctx->kernels_last++;
+        const int per_grid = std::max(1, std::min(256, 2 * ctx->n_sms / std::max(1, n)));
+        for (int j = 0; j < k; j++) {
+            ga.round = j;
+            dk::k_greedy_round<<<n * per_grid, 256, 0, ctx->stream>>>(ga);
+            CU(cudaGetLastError());
+        }
+        dk::k_greedy_emit<<<(n * k + 127) / 128, 128, 0, ctx->stream>>>(ga);
+        CU(cudaGetLastError());
+        ctx->kernels_last += k + 2;
     }
     return DOCK_OK;
 }
@@ -671,7 +681,7 @@ void dock_destroy(dock_ctx* ctx)
     cudaSetDevice(ctx->device);
     if (ctx->stream) cudaStreamSynchronize(ctx->stream);
     DevBuf* bufs[] = {&ctx->xyz, &ctx->coef, &ctx->off, &ctx->rot, &ctx->Lw, &ctx->T, &ctx->mu, &ctx->cnt,
-                      &ctx->cand, &ctx->poses, &ctx->fb_list, &ctx->grid, &ctx->slots, &ctx->units, &ctx->Lw_fb};
+                      &ctx->cand, &ctx->poses, &ctx->fb_list, &ctx->grid, &ctx->slots, &ctx->units, &ctx->Lw_fb, &ctx->picks};
     for (DevBuf* b : bufs)
         if (b->p) cudaFree(b->p);
     if (ctx->d_rec) cudaFree(ctx->d_rec);

@@ -10,7 +10,7 @@
 //                        8 rotations), fused weighted sum, per-warp top-32 lists
 //                        (GRID=false) or a score-grid epilogue (GRID=true)
 //   k_merge          a6  per-rotation greedy best-then-exclude over candidates
-//   k_greedy_grid    a6' exact greedy over a full score grid (fallback)
+//   k_greedy_round   a6' exact greedy over full score grids (fallback)
 #pragma once
 #include <cuda.h>
 #include <cuda_runtime.h>
@@ -619,62 +619,69 @@ __global__ void k_merge(MergeArgs a)
 struct GreedyArgs {
     const float* grid;          // [n][nz][ny][nx]  (slot order of this fallback chunk)
     const int* slots;           // output slot of each grid
-    int n, k, rho, n_rot;
+    unsigned long long* picks;  // [n][k] picks so far (KEY_MAX = none)
+    int n, k, rho, n_rot, round;
     int nx, ny, nz;
     long long unit_begin;
     void* poses;
 };
 
-// One CTA per grid: the paper's scoring + filtering loop with the whole CTA
-// scanning the N^3 cells for the best available key each round.
-__global__ void __launch_bounds__(1024) k_greedy_grid(GreedyArgs a)
+// One round j of the paper's best-then-exclude loop over full score grids,
+// spread over many CTAs per grid: every thread scans a strided share of the N^3 cells for
+// the best key that is farther than rho from picks 0..j-1, and the warp minima are combined
+// with one 64-bit atomicMin per warp into picks[g][j].
+__global__ void k_greedy_round(GreedyArgs a)
 {
-    __shared__ unsigned long long red[32];
-    __shared__ unsigned long long picks[32];
-    const int gi = blockIdx.x;
-    if (gi >= a.n) return;
+    const int ctas_per_grid = gridDim.x / a.n;
+    const int gi = blockIdx.x / ctas_per_grid, part = blockIdx.x % ctas_per_grid;
     const float* S = a.grid + static_cast<size_t>(gi) * a.nx * a.ny * a.nz;
     const uint32_t ncell = static_cast<uint32_t>(a.nx) * a.ny * a.nz;
-    int np = 0;
-    for (int j = 0; j < a.k; j++) {
-        unsigned long long best = KEY_MAX;
-        for (uint32_t t = threadIdx.x; t < ncell; t += blockDim.x) {
-            const unsigned long long key = make_key(S[t], t);
-            if (key >= best) continue;
-            bool ok = true;
-            for (int q = 0; q < j; q++)
-                ok = ok && (cheb_cyc(t, static_cast<uint32_t>(picks[q] & 0xffffffffu), a.nx, a.ny, a.nz) > a.rho);
-            if (ok) best = key;
-        }
-        best = warp_min_u64(best);
-        if ((threadIdx.x & 31) == 0) red[threadIdx.x >> 5] = best;
-        __syncthreads();
-        if (threadIdx.x < 32) {
-            unsigned long long v = threadIdx.x < (blockDim.x >> 5) ? red[threadIdx.x] : KEY_MAX;
-            v = warp_min_u64(v);
-            if (threadIdx.x == 0) picks[j] = v;
-        }
-        __syncthreads();
-        if (picks[j] == KEY_MAX) break;
-        np++;
+    unsigned long long* pk = a.picks + static_cast<size_t>(gi) * a.k;
+    const int j = a.round;
+    uint32_t prev[32];
+    for (int q = 0; q < j; q++) prev[q] = static_cast<uint32_t>(pk[q] & 0xffffffffu);
+    if (j > 0 && pk[j - 1] == KEY_MAX) return;   // fewer than j picks possible
+    unsigned long long best = KEY_MAX;
+    const uint32_t stride = static_cast<uint32_t>(ctas_per_grid) * blockDim.x;
+    for (uint32_t t = part * blockDim.x + threadIdx.x; t < ncell; t += stride) {
+        const unsigned long long key = make_key(S[t], t);
+        if (key >= best) continue;
+        bool ok = true;
+        for (int q = 0; q < j; q++) ok = ok && (cheb_cyc(t, prev[q], a.nx, a.ny, a.nz) > a.rho);
+        if (ok) best = key;
     }
+    best = warp_min_u64(best);
+    if ((threadIdx.x & 31) == 0 && best != KEY_MAX) atomicMin(&pk[j], best);
+}
+
+// Write the fallback poses (flag DOCK_POSE_FALLBACK) once all rounds are done.
+__global__ void k_greedy_emit(GreedyArgs a)
+{
+    const int i = blockIdx.x * blockDim.x + threadIdx.x;
+    if (i >= a.n * a.k) return;
+    const int gi = i / a.k, j = i % a.k;
+    const unsigned long long key = a.picks[static_cast<size_t>(gi) * a.k + j];
     const int slot = a.slots[gi];
     const long long unit = a.unit_begin + slot;
-    PoseOut* out = reinterpret_cast<PoseOut*>(a.poses) + static_cast<size_t>(slot) * a.k;
-    for (int j = threadIdx.x; j < a.k; j += blockDim.x) {
-        PoseOut po;
-        po.rot = static_cast<int32_t>(unit % a.n_rot);
-        if (j < np) {
-            po.t_lin = static_cast<int32_t>(picks[j] & 0xffffffffu);
-            po.score = unord_f32(static_cast<uint32_t>(picks[j] >> 32));
-            po.flags = 1u;
-        } else {
-            po.t_lin = -1;
-            po.score = __int_as_float(0x7fc00000);
-            po.flags = 3u;
-        }
-        out[j] = po;
+    PoseOut po;
+    po.rot = static_cast<int32_t>(unit % a.n_rot);
+    if (key != KEY_MAX) {
+        po.t_lin = static_cast<int32_t>(key & 0xffffffffu);
+        po.score = unord_f32(static_cast<uint32_t>(key >> 32));
+        po.flags = 1u;
+    } else {
+        po.t_lin = -1;
+        po.score = __int_as_float(0x7fc00000);
+        po.flags = 3u;
     }
+    reinterpret_cast<PoseOut*>(a.poses)[static_cast<size_t>(slot) * a.k + j] = po;
+}
+
+__global__ void k_fill_u64(unsigned long long* p, size_t n, unsigned long long v)
+{
+    for (size_t i = blockIdx.x * static_cast<size_t>(blockDim.x) + threadIdx.x; i < n;
+         i += static_cast<size_t>(gridDim.x) * blockDim.x)
+        p[i] = v;
 }
 
 // ------------------------------------------------------------------ per-call state reset

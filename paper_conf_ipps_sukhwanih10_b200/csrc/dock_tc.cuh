@@ -31,9 +31,9 @@ constexpr int ROT = 128;        // rotations per block (MMA M)
 constexpr int NT = 128;         // translations per row (MMA N)
 constexpr int NEPI = 8;         // epilogue warps (2 per TMEM lane quarter)
 constexpr int NTHREADS = (2 + NEPI) * 32;
-constexpr int WSTAGES = 8;      // weight ring depth
+constexpr int WSTAGES = 16;     // weight ring depth (16 x 4 KB covers the L2 latency)
 constexpr int WCHUNK = 2 * ROT * 16;   // bytes of one K-step of A (2 K-chunks x 128 rotations x 16 B)
-constexpr int LIST = 16;        // per-thread candidate list
+constexpr int LIST = 32;        // per-thread candidate list (exact top-LIST keys of one rotation)
 
 struct TcArgs {
     int nx, ny, nz;
@@ -267,14 +267,24 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                             for (int j = 0; j < 32; j++)
                                 if (x0 + c0 + j < a.nx) out[c0 + j] = __uint_as_float(v[j]);
                         } else {
+                            // fast check: one FMNMX per value; the insertion path is rare after warm-up
+                            float mn = __uint_as_float(v[0]);
 #pragma unroll
-                            for (int j = 0; j < 32; j++) {
-                                const float sv = __uint_as_float(v[j]);
-                                if (sv <= th && x0 + c0 + j < a.nx) {
-                                    const unsigned long long key = dk::make_key(sv, tbase + c0 + j);
-                                    if (key < lst[LIST - 1]) {
-                                        list_insert(lst, key);
-                                        th = dk::key_score_bound(static_cast<uint32_t>(lst[LIST - 1] >> 32));
+                            for (int j = 1; j < 32; j++) mn = fminf(mn, __uint_as_float(v[j]));
+                            if (mn <= th) {
+                                float vv[32];
+#pragma unroll
+                                for (int j = 0; j < 32; j++) vv[j] = __uint_as_float(v[j]);
+                                const int jmax = min(32, a.nx - x0 - c0);
+#pragma unroll 1
+                                for (int j = 0; j < jmax; j++) {
+                                    const float sv = vv[j];
+                                    if (sv <= th) {
+                                        const unsigned long long key = dk::make_key(sv, tbase + c0 + j);
+                                        if (key < lst[LIST - 1]) {
+                                            list_insert(lst, key);
+                                            th = dk::key_score_bound(static_cast<uint32_t>(lst[LIST - 1] >> 32));
+                                        }
                                     }
                                 }
                             }
@@ -287,28 +297,36 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
             }
             if constexpr (!GRID) {
                 if (rot_ok) {
-                    // bound: k list entries pairwise farther than 2*rho apart
+                    // bound: k list entries pairwise farther than 2*rho apart.
+                    // Loops over the register list are fully unrolled (static indices keep it in registers).
                     unsigned long long Tw = KEY_MAX;
-                    uint32_t chosen[dk::RB * 4];
+                    uint32_t chosen[32];
                     int nc = 0;
-                    for (int i = 0; i < LIST && nc < a.k; i++) {
-                        if (lst[i] == KEY_MAX) break;
-                        const uint32_t t = static_cast<uint32_t>(lst[i] & 0xffffffffu);
-                        bool far = true;
-                        for (int c = 0; c < nc; c++)
-                            far = far && dk::cheb_cyc(t, chosen[c], a.nx, a.ny, a.nz) > 2 * a.rho;
-                        if (far) {
-                            chosen[nc++] = t;
-                            if (nc == a.k) Tw = lst[i];
+#pragma unroll
+                    for (int i = 0; i < LIST; i++) {
+                        const unsigned long long key = lst[i];
+                        if (key != KEY_MAX && nc < a.k) {
+                            const uint32_t t = static_cast<uint32_t>(key & 0xffffffffu);
+                            bool far = true;
+                            for (int c = 0; c < nc; c++)
+                                far = far && dk::cheb_cyc(t, chosen[c], a.nx, a.ny, a.nz) > 2 * a.rho;
+                            if (far) {
+                                chosen[nc] = t;
+                                nc++;
+                                if (nc == a.k) Tw = key;
+                            }
                         }
                     }
                     const unsigned long long old = atomicMin(&a.T[slot], Tw);
                     const unsigned long long Tn = old < Tw ? old : Tw;
                     atomicMin(&a.mu[slot], lst[LIST - 1]);
+#pragma unroll
                     for (int i = 0; i < LIST; i++) {
-                        if (lst[i] == KEY_MAX || lst[i] > Tn) break;
-                        const unsigned pos = atomicAdd(&a.cnt[slot], 1u);
-                        if (pos < static_cast<unsigned>(a.cap)) a.cand[static_cast<size_t>(slot) * a.cap + pos] = lst[i];
+                        const unsigned long long key = lst[i];
+                        if (key != KEY_MAX && key <= Tn) {
+                            const unsigned pos = atomicAdd(&a.cnt[slot], 1u);
+                            if (pos < static_cast<unsigned>(a.cap)) a.cand[static_cast<size_t>(slot) * a.cap + pos] = key;
+                        }
                     }
                 }
             }

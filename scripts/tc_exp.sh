@@ -1,0 +1,17 @@
+#!/bin/bash
+# tcgen05 engine experiments: Q=4/NBUF=1 vs Q=2/NBUF=2, then one ncu capture of k_corr_tc.
+set -u
+mkdir -p gpurun_out
+TAG=${1:-x}
+B="python bench.py --steps 3 --warmup 2 --no-e2e --no-cpu-baseline --no-alt --engine tc"
+G='"value": [0-9.]*\|"launch_ms": [0-9.]*\|"executed_frac": [0-9.]*\|fallback_rotations": [0-9]*'
+echo "== Q4"; timeout 300 $B > gpurun_out/tc_${TAG}_q4.log 2>&1; grep -o "$G" gpurun_out/tc_${TAG}_q4.log
+echo "== Q2"; DOCK_TC_Q=2 timeout 300 $B > gpurun_out/tc_${TAG}_q2.log 2>&1; grep -o "$G" gpurun_out/tc_${TAG}_q2.log
+if [ "${NCU:-1}" = "1" ]; then
+timeout 900 ncu --set full --clock-control none --import-source on -k regex:k_corr_tc -s 1 -c 1 \
+    -o gpurun_out/tc_${TAG} -f $B > gpurun_out/tc_${TAG}_ncu.log 2>&1
+echo "ncu rc=$?"
+ncu -i gpurun_out/tc_${TAG}.ncu-rep --page raw --csv > gpurun_out/tc_${TAG}_raw.csv 2>/dev/null
+ncu -i gpurun_out/tc_${TAG}.ncu-rep --page source --csv > gpurun_out/tc_${TAG}_source.csv 2>/dev/null
+ncu -i gpurun_out/tc_${TAG}.ncu-rep --page details --csv > gpurun_out/tc_${TAG}_details.csv 2>/dev/null
+fi
