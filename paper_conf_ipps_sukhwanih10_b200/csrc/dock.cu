@@ -35,7 +35,8 @@ struct DevBuf {
 struct TcPlan {                // per-probe-size plan of the tcgen05 engine
     bool ok = false;
     CUtensorMap tmap;
-    int TXB = 0, TYB = 0, TZB = 0, box_bytes = 0, rec_stage_bytes = 0, n_rec_stages = 0, smem = 0, nsteps = 0;
+    int TXB = 0, TYB = 0, TZB = 0, box_bytes = 0, rec_stage_bytes = 0, n_rec_stages = 0, smem = 0, nsteps = 0,
+        wstages = 0;
 };
 
 struct MPlan {                 // per-probe-size launch plan
@@ -277,11 +278,13 @@ dock_status make_tc_plan(dock_ctx* ctx, int m)
     pl.box_bytes = 16 * pl.TXB * pl.TYB * pl.TZB;
     pl.rec_stage_bytes = round_up(ctx->tc_Gch * pl.box_bytes, 1024);
     pl.nsteps = ctx->tc_Gch * 2 * m * m * ((m + 1) / 2);
-    const int ring = tc::WSTAGES * tc::WCHUNK;
     const int budget = kSmemLimit - 2048;   // static shared memory (barriers) and slack
-    if (2 * pl.rec_stage_bytes + ring <= budget) pl.n_rec_stages = 2;
-    else if (pl.rec_stage_bytes + ring <= budget) pl.n_rec_stages = 1;
+    const int min_ring = 4 * tc::WCHUNK;
+    if (2 * pl.rec_stage_bytes + min_ring <= budget) pl.n_rec_stages = 2;
+    else if (pl.rec_stage_bytes + min_ring <= budget) pl.n_rec_stages = 1;
     else return DOCK_OK;                    // this m is not eligible for the tensor-core engine
+    pl.wstages = std::min(tc::WSTAGES, (budget - pl.n_rec_stages * pl.rec_stage_bytes) / tc::WCHUNK);
+    const int ring = pl.wstages * tc::WCHUNK;
     // >= 116 KB keeps one CTA per SM: every CTA allocates all 512 TMEM columns
     pl.smem = std::max(pl.n_rec_stages * pl.rec_stage_bytes + ring, 116 * 1024);
     auto fn = encode_fn();
@@ -612,6 +615,7 @@ tc::TcArgs tc_args(dock_ctx* ctx, int m, int n_slots, int G, const unsigned char
     a.box_bytes = tp.box_bytes;
     a.rec_stage_bytes = tp.rec_stage_bytes;
     a.n_rec_stages = tp.n_rec_stages;
+    a.wstages = tp.wstages;
     return a;
 }
 

@@ -31,7 +31,7 @@ constexpr int ROT = 128;        // rotations per block (MMA M)
 constexpr int NT = 128;         // translations per row (MMA N)
 constexpr int NEPI = 8;         // epilogue warps (2 per TMEM lane quarter)
 constexpr int NTHREADS = (2 + NEPI) * 32;
-constexpr int WSTAGES = 16;     // weight ring depth (16 x 4 KB covers the L2 latency)
+constexpr int WSTAGES = 16;     // max weight ring depth (runtime a.wstages <= 16; 16 x 4 KB covers the L2 latency)
 constexpr int WCHUNK = 2 * ROT * 16;   // bytes of one K-step of A (2 K-chunks x 128 rotations x 16 B)
 constexpr int LIST = 32;        // per-thread candidate list (exact top-LIST keys of one rotation)
 
@@ -46,6 +46,7 @@ struct TcArgs {
     int box_bytes;              // one channel group's receptor box
     int rec_stage_bytes;        // G_ch * box_bytes rounded to 1024
     int n_rec_stages;           // 1 or 2
+    int wstages;                // weight ring depth (4..WSTAGES)
     // top-k
     int k, rho, cap;
     unsigned long long* T;
@@ -115,6 +116,15 @@ __device__ __forceinline__ void tma_load_5d(void* dst, const CUtensorMap* map, i
         : "memory");
 }
 
+__device__ __forceinline__ bool elect_one()
+{
+    uint32_t pred = 0;
+    asm volatile(
+        "{\n\t.reg .pred P;\n\telect.sync _|P, 0xffffffff;\n\tselp.u32 %0, 1, 0, P;\n\t}\n"
+        : "=r"(pred));
+    return pred != 0;
+}
+
 // Sorted (ascending) per-thread key list, fully unrolled insertion.
 __device__ __forceinline__ void list_insert(unsigned long long (&L)[LIST], unsigned long long key)
 {
@@ -154,7 +164,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
             dk::mbar_init(&rec_full[i], 1);
             dk::mbar_init(&rec_empty[i], 1);
         }
-        for (int i = 0; i < WSTAGES; i++) {
+        for (int i = 0; i < a.wstages; i++) {
             dk::mbar_init(&w_full[i], 1);
             dk::mbar_init(&w_empty[i], 1);
         }
@@ -176,63 +186,89 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
 
     if (n_tiles > 0) {
         if (warp == 0) {
-            // ------------------------------------------------ TMA producer
-            if (lane == 0) {
-                dk::prefetch_tmap(&tmap);
-                const unsigned char* wsrc = a.W + static_cast<size_t>(block) * a.nsteps * WCHUNK;
-                int wi = 0;
-                for (int ti = 0; ti < n_tiles; ti++) {
-                    const int tile = tile_begin + ti;
-                    const int rs = ti % a.n_rec_stages, ruse = ti / a.n_rec_stages;
-                    if (ruse > 0) dk::mbar_wait(&rec_empty[rs], (ruse - 1) & 1);
-                    const int tx = tile % a.ntx, ty = (tile / a.ntx) % a.nty, tz = tile / (a.ntx * a.nty);
-                    unsigned char* rdst = rec_smem + static_cast<size_t>(rs) * a.rec_stage_bytes;
+            // ------------------------------------------------ TMA producer (warp-converged, one elected lane)
+            if (elect_one()) dk::prefetch_tmap(&tmap);
+            const unsigned char* wsrc = a.W + static_cast<size_t>(block) * a.nsteps * WCHUNK;
+            int ws = 0, wph = 0;                  // weight ring slot / phase
+            int wuse = 0;
+            for (int ti = 0; ti < n_tiles; ti++) {
+                const int tile = tile_begin + ti;
+                const int rs = ti % a.n_rec_stages, ruse = ti / a.n_rec_stages;
+                if (ruse > 0) dk::mbar_wait(&rec_empty[rs], (ruse - 1) & 1);
+                const int tx = tile % a.ntx, ty = (tile / a.ntx) % a.nty, tz = tile / (a.ntx * a.nty);
+                unsigned char* rdst = rec_smem + static_cast<size_t>(rs) * a.rec_stage_bytes;
+                if (elect_one()) {
                     dk::mbar_arrive_expect_tx(&rec_full[rs], a.G_ch * a.box_bytes);
                     for (int g = 0; g < a.G_ch; g++)
                         tma_load_5d(rdst + static_cast<size_t>(g) * a.box_bytes, &tmap, 0, tx * NT, ty * Q, tz, g,
                                     &rec_full[rs]);
-                    for (int s = 0; s < a.nsteps; s++, wi++) {
-                        const int ws = wi % WSTAGES, wuse = wi / WSTAGES;
-                        if (wuse > 0) dk::mbar_wait(&w_empty[ws], (wuse - 1) & 1);
+                }
+                __syncwarp();
+                for (int s = 0; s < a.nsteps; s++) {
+                    if (wuse >= a.wstages) dk::mbar_wait(&w_empty[ws], wph ^ 1);
+                    if (elect_one()) {
                         dk::mbar_arrive_expect_tx(&w_full[ws], WCHUNK);
                         dk::bulk_load(w_smem + static_cast<size_t>(ws) * WCHUNK, wsrc + static_cast<size_t>(s) * WCHUNK,
                                       WCHUNK, &w_full[ws]);
                     }
+                    __syncwarp();
+                    wuse++;
+                    if (++ws == a.wstages) {
+                        ws = 0;
+                        wph ^= 1;
+                    }
                 }
             }
         } else if (warp == 1) {
-            // ------------------------------------------------ MMA issuer (one thread)
-            if (lane == 0) {
-                constexpr uint32_t idesc = umma_idesc(ROT, NT);
-                const uint32_t rec0 = dk::smem_u32(rec_smem), w0 = dk::smem_u32(w_smem);
-                int wi = 0;
-                for (int ti = 0; ti < n_tiles; ti++) {
-                    const int rs = ti % a.n_rec_stages, ruse = ti / a.n_rec_stages;
-                    const int buf = ti % NBUF, buse = ti / NBUF;
-                    dk::mbar_wait(&rec_full[rs], ruse & 1);
-                    if (buse > 0) dk::mbar_wait(&tm_empty[buf], (buse - 1) & 1);
-                    tc_fence_after();
-                    const uint32_t rbase = rec0 + rs * a.rec_stage_bytes;
-                    for (int s = 0; s < a.nsteps; s++, wi++) {
-                        const int ws = wi % WSTAGES, wuse = wi / WSTAGES;
-                        dk::mbar_wait(&w_full[ws], wuse & 1);
-                        tc_fence_after();
-                        // step s -> (g, pass, vz, vy, vxp)
-                        const int vxp = s % MXP, vy = (s / MXP) % M, vz = (s / (MXP * M)) % M;
-                        const int g = s / (MXP * M * M * 2);
-                        const uint64_t da = umma_desc(w0 + ws * WCHUNK, ROT * 16, 128);
-                        const uint32_t bq =
-                            rbase + g * a.box_bytes + ((vz * a.TYB + vy) * a.TXB + 2 * vxp) * 16;
+            // ------------------------------------------------ MMA issuer (warp-converged, one elected lane)
+            constexpr uint32_t idesc = umma_idesc(ROT, NT);
+            const uint32_t rec0 = dk::smem_u32(rec_smem), w0 = dk::smem_u32(w_smem);
+            const uint64_t dA0 = umma_desc(w0, ROT * 16, 128);   // + (slot offset >> 4)
+            const uint64_t dB0 = umma_desc(rec0, 16, 128);       // + (voxel offset >> 4)
+            const uint32_t row16 = static_cast<uint32_t>(a.TXB) * 16u;
+            int ws = 0, wph = 0;
+            for (int ti = 0; ti < n_tiles; ti++) {
+                const int rs = ti % a.n_rec_stages, ruse = ti / a.n_rec_stages;
+                const int buf = ti % NBUF, buse = ti / NBUF;
+                dk::mbar_wait(&rec_full[rs], ruse & 1);
+                if (buse > 0) dk::mbar_wait(&tm_empty[buf], (buse - 1) & 1);
+                tc_fence_after();
+                const uint32_t dcol = tmem + static_cast<uint32_t>(buf * Q * NT);
+                uint32_t acc = 0;
+                for (int g = 0; g < a.G_ch; g++) {
+                    const uint32_t gofs = static_cast<uint32_t>(rs * a.rec_stage_bytes + g * a.box_bytes);
+                    for (int pass = 0; pass < 2; pass++) {
+                        for (int vz = 0; vz < M; vz++) {
+                            for (int vy = 0; vy < M; vy++) {
+                                const uint32_t rowofs = gofs + static_cast<uint32_t>(vz * a.TYB + vy) * row16;
 #pragma unroll
-                        for (int q = 0; q < Q; q++) {
-                            const uint64_t db = umma_desc(bq + q * a.TXB * 16, 16, 128);
-                            umma_bf16(tmem + (buf * Q + q) * NT, da, db, idesc, s > 0 ? 1u : 0u);
+                                for (int vxp = 0; vxp < MXP; vxp++) {
+                                    dk::mbar_wait(&w_full[ws], wph);
+                                    tc_fence_after();
+                                    if (elect_one()) {
+                                        const uint64_t da = dA0 + ((static_cast<uint32_t>(ws) * WCHUNK) >> 4);
+                                        const uint64_t db = dB0 + ((rowofs + vxp * 32u) >> 4);
+#pragma unroll
+                                        for (int q = 0; q < Q; q++)
+                                            umma_bf16(dcol + q * NT, da, db + ((q * row16) >> 4), idesc, acc);
+                                        umma_commit(&w_empty[ws]);
+                                    }
+                                    __syncwarp();
+                                    acc = 1;
+                                    if (++ws == a.wstages) {
+                                        ws = 0;
+                                        wph ^= 1;
+                                    }
+                                }
+                            }
                         }
-                        umma_commit(&w_empty[ws]);
                     }
+                }
+                if (elect_one()) {
                     umma_commit(&tm_full[buf]);
                     umma_commit(&rec_empty[rs]);
                 }
+                __syncwarp();
             }
         } else {
             // ------------------------------------------------ epilogue warps
