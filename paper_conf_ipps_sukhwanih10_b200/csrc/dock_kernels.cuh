@@ -438,47 +438,40 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr(const __grid_constant__ CU
                 }
             }
         } else {
-            // fast check: any value at or below its rotation's current 32nd-best score?
+            // fast check: which rotations have a value at or below their warp list's 32nd-best score?
             unsigned vmask = 0;
 #pragma unroll
             for (int x = 0; x < XT; x++) vmask |= (row_ok && tx0 + x < a.g.nx) ? (1u << x) : 0u;
-            bool any = false;
+            unsigned pend = 0;
 #pragma unroll
             for (int r = 0; r < RB; r++) {
                 const float th = key_score_bound(static_cast<uint32_t>(shfl_u64(lst[r], 31) >> 32));
-                if (r < nb) {
+                bool any = false;
 #pragma unroll
-                    for (int x = 0; x < XT; x++) any |= ((vmask >> x) & 1u) && (acc[r][x] <= th);
-                }
+                for (int x = 0; x < XT; x++) any |= ((vmask >> x) & 1u) && (acc[r][x] <= th);
+                pend |= (any && r < nb) ? (1u << r) : 0u;
             }
-            if (__any_sync(FULL, any)) {
-                // slow path: rotate the register blocks so the body is written once (acc is dead after)
-#pragma unroll 1
-                for (int rr = 0; rr < RB; rr++) {
-                    if (rr < nb) {
-                        unsigned long long th = shfl_u64(lst[0], 31);
+            const unsigned wpend = __reduce_or_sync(FULL, pend);
+            if (wpend) {
+                // slow path, only for the rotations that need it (warp-uniform branches)
+#pragma unroll
+                for (int r = 0; r < RB; r++) {
+                    if ((wpend >> r) & 1u) {
+                        unsigned long long th = shfl_u64(lst[r], 31);
 #pragma unroll
                         for (int x = 0; x < XT; x++) {
                             const unsigned long long key =
-                                ((vmask >> x) & 1u) ? make_key(acc[0][x], tbase + x) : KEY_MAX;
+                                ((vmask >> x) & 1u) ? make_key(acc[r][x], tbase + x) : KEY_MAX;
                             unsigned m = __ballot_sync(FULL, key < th);
                             while (m) {
                                 const int src = __ffs(m) - 1;
-                                warp_list_insert(lst[0], shfl_u64(key, src), lane);
-                                th = shfl_u64(lst[0], 31);
+                                warp_list_insert(lst[r], shfl_u64(key, src), lane);
+                                th = shfl_u64(lst[r], 31);
                                 m &= ~(1u << src);
                                 m &= __ballot_sync(FULL, key < th);
                             }
                         }
                     }
-                    const unsigned long long l0 = lst[0];
-#pragma unroll
-                    for (int r = 0; r < RB - 1; r++) {
-                        lst[r] = lst[r + 1];
-#pragma unroll
-                        for (int x = 0; x < XT; x++) acc[r][x] = acc[r + 1][x];
-                    }
-                    lst[RB - 1] = l0;
                 }
             }
         }

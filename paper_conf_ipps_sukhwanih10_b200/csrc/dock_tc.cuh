@@ -125,6 +125,21 @@ __device__ __forceinline__ bool elect_one()
     return pred != 0;
 }
 
+// v[j] for a runtime j without local memory: binary select tree over the 5 bits of j.
+__device__ __forceinline__ uint32_t select32(const uint32_t (&v)[32], int j)
+{
+    uint32_t l1[16], l2[8], l3[4], l4[2];
+#pragma unroll
+    for (int i = 0; i < 16; i++) l1[i] = (j & 1) ? v[2 * i + 1] : v[2 * i];
+#pragma unroll
+    for (int i = 0; i < 8; i++) l2[i] = (j & 2) ? l1[2 * i + 1] : l1[2 * i];
+#pragma unroll
+    for (int i = 0; i < 4; i++) l3[i] = (j & 4) ? l2[2 * i + 1] : l2[2 * i];
+#pragma unroll
+    for (int i = 0; i < 2; i++) l4[i] = (j & 8) ? l3[2 * i + 1] : l3[2 * i];
+    return (j & 16) ? l4[1] : l4[0];
+}
+
 // Sorted (ascending) per-thread key list, fully unrolled insertion.
 __device__ __forceinline__ void list_insert(unsigned long long (&L)[LIST], unsigned long long key)
 {
@@ -308,13 +323,16 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
 #pragma unroll
                             for (int j = 1; j < 32; j++) mn = fminf(mn, __uint_as_float(v[j]));
                             if (mn <= th) {
-                                float vv[32];
-#pragma unroll
-                                for (int j = 0; j < 32; j++) vv[j] = __uint_as_float(v[j]);
+                                // rare path: bitmask of candidates, each extracted with a 5-level select tree
                                 const int jmax = min(32, a.nx - x0 - c0);
-#pragma unroll 1
-                                for (int j = 0; j < jmax; j++) {
-                                    const float sv = vv[j];
+                                uint32_t msk = 0;
+#pragma unroll
+                                for (int j = 0; j < 32; j++)
+                                    msk |= (__uint_as_float(v[j]) <= th && j < jmax) ? (1u << j) : 0u;
+                                while (msk) {
+                                    const int j = __ffs(msk) - 1;
+                                    msk &= msk - 1;
+                                    const float sv = __uint_as_float(select32(v, j));
                                     if (sv <= th) {
                                         const unsigned long long key = dk::make_key(sv, tbase + c0 + j);
                                         if (key < lst[LIST - 1]) {

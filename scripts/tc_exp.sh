@@ -7,6 +7,7 @@ B="python bench.py --steps 3 --warmup 2 --no-e2e --no-cpu-baseline --no-alt --en
 G='"value": [0-9.]*\|"launch_ms": [0-9.]*\|"executed_frac": [0-9.]*\|fallback_rotations": [0-9]*'
 echo "== Q4"; timeout 300 $B > gpurun_out/tc_${TAG}_q4.log 2>&1; grep -o "$G" gpurun_out/tc_${TAG}_q4.log
 echo "== Q2"; DOCK_TC_Q=2 timeout 300 $B > gpurun_out/tc_${TAG}_q2.log 2>&1; grep -o "$G" gpurun_out/tc_${TAG}_q2.log
+echo "== FFMA"; timeout 300 python bench.py --steps 3 --warmup 2 --no-e2e --no-cpu-baseline --no-alt --engine ffma > gpurun_out/ffma_${TAG}.log 2>&1; grep -o '"value": [0-9.]*\|"launch_ms": [0-9.]*\|"frac": [0-9.]*' gpurun_out/ffma_${TAG}.log
 if [ "${NCU:-1}" = "1" ]; then
 timeout 900 ncu --set full --clock-control none --import-source on -k regex:k_corr_tc -s 1 -c 1 \
     -o gpurun_out/tc_${TAG} -f $B > gpurun_out/tc_${TAG}_ncu.log 2>&1

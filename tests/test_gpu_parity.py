@@ -330,3 +330,16 @@ def test_prod_config_sampled(D, orc, engine):
     units = [0, 1, 499, 500, 3777, 7999] + list(range(137, 8000, 811))
     _, info, _ = _dock_and_validate(D, orc, R, w, probes, rot, c.k, 1, units=units, engine=engine)
     assert info["fallback_last"] <= 80 and info["engine_last"] == engine
+
+
+def test_large_config_sampled(D, orc):
+    """configs[4] shape: 160^3 receptor, 8^3 probe, 22 terms (pairwise-potential channels), k=4, rho=1.
+    A 256-rotation slice of the 70k-rotation set is docked on the GPU (the FFMA engine: the 22-channel
+    tcgen05 receptor box does not fit shared memory); two units are validated against the oracle."""
+    c = g.CONFIGS["large"]
+    R = g.receptor_ftmap_like(c.n, c.P)
+    w = g.weights(c.P)
+    probes = g.probes(1, c.m, c.P)
+    rot = g.rotations(256, seed=3001)
+    _, info, _ = _dock_and_validate(D, orc, R, w, probes, rot, c.k, 1, units=[0, 173])
+    assert info["fallback_last"] <= 4
