@@ -445,10 +445,13 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr(const __grid_constant__ CU
             unsigned pend = 0;
 #pragma unroll
             for (int r = 0; r < RB; r++) {
-                const float th = key_score_bound(static_cast<uint32_t>(shfl_u64(lst[r], 31) >> 32));
-                bool any = false;
+                // exact gate: a strictly better score, or a tie whose t_lin could precede the 32nd key
+                const unsigned long long l31 = shfl_u64(lst[r], 31);
+                const float th = key_score_bound(static_cast<uint32_t>(l31 >> 32));
+                float mn = __int_as_float(0x7f800000);
 #pragma unroll
-                for (int x = 0; x < XT; x++) any |= ((vmask >> x) & 1u) && (acc[r][x] <= th);
+                for (int x = 0; x < XT; x++) mn = ((vmask >> x) & 1u) ? fminf(mn, acc[r][x]) : mn;
+                const bool any = mn < th || (mn == th && tbase < static_cast<uint32_t>(l31 & 0xffffffffu));
                 pend |= (any && r < nb) ? (1u << r) : 0u;
             }
             const unsigned wpend = __reduce_or_sync(FULL, pend);

@@ -295,7 +295,8 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
             unsigned long long lst[LIST];
 #pragma unroll
             for (int i = 0; i < LIST; i++) lst[i] = KEY_MAX;
-            float th = __int_as_float(0x7f800000);
+            float th = __int_as_float(0x7f800000);   // score of the list's last key (+inf while not full)
+            uint32_t th_t = 0xffffffffu;             // t_lin of the list's last key
             for (int ti = 0; ti < n_tiles; ti++) {
                 const int tile = tile_begin + ti;
                 const int buf = ti % NBUF, buse = ti / NBUF;
@@ -322,7 +323,8 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                             float mn = __uint_as_float(v[0]);
 #pragma unroll
                             for (int j = 1; j < 32; j++) mn = fminf(mn, __uint_as_float(v[j]));
-                            if (mn <= th) {
+                            // exact gate: a strictly better score, or a tie that could carry a smaller t_lin
+                            if (mn < th || (mn == th && tbase + c0 < th_t)) {
                                 // rare path: bitmask of candidates, each extracted with a 5-level select tree
                                 const int jmax = min(32, a.nx - x0 - c0);
                                 uint32_t msk = 0;
@@ -338,6 +340,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                                         if (key < lst[LIST - 1]) {
                                             list_insert(lst, key);
                                             th = dk::key_score_bound(static_cast<uint32_t>(lst[LIST - 1] >> 32));
+                                            th_t = static_cast<uint32_t>(lst[LIST - 1] & 0xffffffffu);
                                         }
                                     }
                                 }
