@@ -195,7 +195,9 @@ def roofline(pk, pk_kind, info, c, flops_launch, corr_ms, ms_step, units_local):
         peak = float(pk.get("bf16_tflops", 1590.0))
         mx = (c.m + 1) // 2 * 2
         executed = flops_launch * 4.0 * mx / c.m
-        return {"bound": "tensor", "engine": "tcgen05 bf16x3", "kernel": f"k_corr_tc<{c.m},4,1,false>",
+        v = int(info.get("tc_variant_last", 1)) or 1
+        kname = f"k_corr_tc<{c.m},4,1,1,false>" if v == 1 else f"k_corr_tc<{c.m},2,2,2,false>"
+        return {"bound": "tensor", "engine": f"tcgen05 bf16x3 (variant {v})", "kernel": kname,
                 "achieved": achieved, "peak": peak, "unit": "TFLOP/s", "frac": achieved / peak, "traffic": None,
                 "peak_source": f"bf16 dense tensor peak, burst, MEASURED_PEAKS.json ({pk_kind})",
                 "executed_tensor_tflops": executed / (corr_ms / 1000.0) / 1e12,

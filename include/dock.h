@@ -135,7 +135,9 @@ typedef enum {
     DOCK_TUNE_REGIONS = 1,        /* translation regions per rotation batch (0 = auto) */
     DOCK_TUNE_FORCE_FALLBACK = 2, /* 1 => every rotation takes the exact full-grid fallback (tests) */
     DOCK_TUNE_CAND_CAP = 3,       /* candidates kept per rotation before overflow fallback (>= 32) */
-    DOCK_TUNE_ENGINE = 4          /* correlation engine: 0 auto (tcgen05 when eligible), 1 FP32 FFMA, 2 tcgen05 */
+    DOCK_TUNE_ENGINE = 4,         /* correlation engine: 0 auto (tcgen05 when eligible), 1 FP32 FFMA, 2 tcgen05 */
+    DOCK_TUNE_TC_VARIANT = 5      /* tcgen05 tiling: 0 auto, 1 = 4 rows x 1 TMEM buffer, 2 = 2 rows x 2 buffers on a
+                                     CTA pair with multicast weight streaming */
 } dock_tune_key;
 
 dock_status dock_set_tuning(dock_ctx* ctx, int key, int64_t value);
@@ -155,6 +157,7 @@ typedef struct {
     int n_sms;                 /* multiprocessors of the context's device */
     int engine_last;           /* engine of the last correlation: 1 FP32 FFMA, 2 tcgen05 bf16x3 */
     int tc_available;          /* 1 if the tcgen05 engine is available for m_max */
+    int tc_variant_last;       /* tcgen05 variant of the last correlation (1 or 2), 0 if FFMA */
 } dock_info;
 
 dock_status dock_get_info(const dock_ctx* ctx, dock_info* info);

@@ -10,7 +10,7 @@ from .dock import (  # noqa: F401
     dock_probe_batch, dock_score_grid, dock_set_tuning, dock_voxelize, poses_from_device,
 )
 from ._native import (  # noqa: F401
-    DOCK_MAX_K, DOCK_MAX_M, DOCK_MAX_TERMS, DOCK_POSE_FALLBACK, DOCK_TUNE_CAND_CAP, DOCK_TUNE_ENGINE,
+    DOCK_MAX_K, DOCK_MAX_M, DOCK_MAX_TERMS, DOCK_POSE_FALLBACK, DOCK_TUNE_CAND_CAP, DOCK_TUNE_ENGINE, DOCK_TUNE_TC_VARIANT,
     DOCK_TUNE_FORCE_FALLBACK, DOCK_TUNE_REGIONS, EXPORTS, LIB_PATH,
 )
 from . import parallel  # noqa: F401,E402

@@ -22,6 +22,7 @@ DOCK_TUNE_REGIONS = 1
 DOCK_TUNE_FORCE_FALLBACK = 2
 DOCK_TUNE_CAND_CAP = 3
 DOCK_TUNE_ENGINE = 4
+DOCK_TUNE_TC_VARIANT = 5
 
 STATUS_NAMES = {0: "DOCK_OK", -1: "DOCK_E_INVALID_ARG", -2: "DOCK_E_UNSUPPORTED",
                 -3: "DOCK_E_PROBE_OUTSIDE_GRID", -4: "DOCK_E_BAD_ROTATION", -5: "DOCK_E_CUDA",
@@ -48,7 +49,8 @@ class dock_info(C.Structure):
                 ("cand_max_last", C.c_int64), ("kernels_last", C.c_int64), ("rot_batch", C.c_int),
                 ("x_per_thread", C.c_int), ("padded_x", C.c_int), ("padded_y", C.c_int),
                 ("padded_z", C.c_int), ("l2_bytes", C.c_double), ("corr_ms_last", C.c_double),
-                ("n_sms", C.c_int), ("engine_last", C.c_int), ("tc_available", C.c_int)]
+                ("n_sms", C.c_int), ("engine_last", C.c_int), ("tc_available", C.c_int),
+                ("tc_variant_last", C.c_int)]
 
 
 EXPORTS = ["dock_init", "dock_probe", "dock_probe_batch", "dock_score_grid", "dock_voxelize",

@@ -65,10 +65,11 @@ struct dock_ctx {
     // tcgen05 engine
     int engine = 0;            // DOCK_TUNE_ENGINE: 0 auto, 1 FFMA, 2 tensor cores
     int engine_last = 0;
-    int tc_q = 4;              // translation rows per TMEM buffer (NBUF = 4 / tc_q)
+    int tc_variant = 0;        // DOCK_TUNE_TC_VARIANT: 0 auto, 1 (Q4, 1 TMEM buffer), 2 (Q2, 2 buffers, CTA pair)
+    int tc_variant_last = 0;
     uint16_t* d_rec_tc = nullptr;
-    int tc_Gch = 0, tc_ntx = 0, tc_nty = 0, tc_ntz = 0, tc_ntiles = 0, tc_Xp = 0, tc_Yp = 0, tc_Zp = 0;
-    TcPlan tcplan[DOCK_MAX_M + 1];
+    int tc_Gch = 0, tc_ntx = 0, tc_ntz = 0, tc_Xp = 0, tc_Yp = 0, tc_Zp = 0;
+    TcPlan tcplan[3][DOCK_MAX_M + 1];   // [variant][m]
     DevBuf Wtc;
     // per-call scratch (grow-only)
     DevBuf xyz, coef, off, rot, Lw, T, mu, cnt, cand, poses, fb_list, grid, slots, units, Lw_fb, picks;
@@ -267,13 +268,18 @@ cudaError_t launch_corr(int m, const MPlan& pl, const dk::CorrArgs& a, int grid,
 }
 
 int tc_txb(int m) { return tc::NT + (m + 1) / 2 * 2 - 1; }
+// tcgen05 variants: 1 = Q4 rows x 1 TMEM buffer, single CTA; 2 = Q2 rows x 2 buffers, CTA pair + multicast.
+inline int tc_q(int v) { return v == 1 ? 4 : 2; }
+inline int tc_cl(int v) { return v == 1 ? 1 : 2; }
+inline int tc_nty(const dock_ctx* c, int v) { return (c->ny + tc_q(v) - 1) / tc_q(v); }
+inline int tc_ntiles(const dock_ctx* c, int v) { return c->tc_ntx * tc_nty(c, v) * c->tc_ntz; }
 
-dock_status make_tc_plan(dock_ctx* ctx, int m)
+dock_status make_tc_plan(dock_ctx* ctx, int m, int v)
 {
-    TcPlan& pl = ctx->tcplan[m];
+    TcPlan& pl = ctx->tcplan[v][m];
     if (pl.ok || !ctx->d_rec_tc) return DOCK_OK;
     pl.TXB = tc_txb(m);
-    pl.TYB = ctx->tc_q + m - 1;
+    pl.TYB = tc_q(v) + m - 1;
     pl.TZB = m;
     pl.box_bytes = 16 * pl.TXB * pl.TYB * pl.TZB;
     pl.rec_stage_bytes = round_up(ctx->tc_Gch * pl.box_bytes, 1024);
@@ -302,34 +308,74 @@ dock_status make_tc_plan(dock_ctx* ctx, int m)
     return DOCK_OK;
 }
 
-template <int M, int Q, bool GRID>
+template <int M, int Q, int NBUF, int CL, bool GRID>
 cudaError_t launch_tc_t(const TcPlan& pl, const tc::TcArgs& a, int grid, cudaStream_t st)
 {
-    auto kern = tc::k_corr_tc<M, Q, 4 / Q, GRID>;
+    auto kern = tc::k_corr_tc<M, Q, NBUF, CL, GRID>;
     cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, pl.smem);
     if (e != cudaSuccess) return e;
-    kern<<<grid, tc::NTHREADS, pl.smem, st>>>(pl.tmap, a);
+    if constexpr (CL == 1) {
+        kern<<<grid, tc::NTHREADS, pl.smem, st>>>(pl.tmap, a);
+    } else {
+        cudaLaunchConfig_t cfg{};
+        cfg.gridDim = dim3(grid);
+        cfg.blockDim = dim3(tc::NTHREADS);
+        cfg.dynamicSmemBytes = pl.smem;
+        cfg.stream = st;
+        cudaLaunchAttribute at[1];
+        at[0].id = cudaLaunchAttributeClusterDimension;
+        at[0].val.clusterDim.x = CL;
+        at[0].val.clusterDim.y = 1;
+        at[0].val.clusterDim.z = 1;
+        cfg.attrs = at;
+        cfg.numAttrs = 1;
+        e = cudaLaunchKernelEx(&cfg, kern, pl.tmap, a);
+        if (e != cudaSuccess) return e;
+    }
     return cudaGetLastError();
 }
 
-template <bool GRID>
-cudaError_t launch_tc(int m, int q, const TcPlan& pl, const tc::TcArgs& a, int grid, cudaStream_t st)
+template <int V, bool GRID>
+cudaError_t launch_tc_v(int m, const TcPlan& pl, const tc::TcArgs& a, int grid, cudaStream_t st)
 {
-    if (q == 2) {
-        if (m == 4) return launch_tc_t<4, 2, GRID>(pl, a, grid, st);
-        return cudaErrorInvalidValue;
-    }
+    constexpr int Q = V == 1 ? 4 : 2, NB = V == 1 ? 1 : 2, CL = V == 1 ? 1 : 2;
     switch (m) {
-        case 1: return launch_tc_t<1, 4, GRID>(pl, a, grid, st);
-        case 2: return launch_tc_t<2, 4, GRID>(pl, a, grid, st);
-        case 3: return launch_tc_t<3, 4, GRID>(pl, a, grid, st);
-        case 4: return launch_tc_t<4, 4, GRID>(pl, a, grid, st);
-        case 5: return launch_tc_t<5, 4, GRID>(pl, a, grid, st);
-        case 6: return launch_tc_t<6, 4, GRID>(pl, a, grid, st);
-        case 7: return launch_tc_t<7, 4, GRID>(pl, a, grid, st);
-        case 8: return launch_tc_t<8, 4, GRID>(pl, a, grid, st);
+        case 1: return launch_tc_t<1, Q, NB, CL, GRID>(pl, a, grid, st);
+        case 2: return launch_tc_t<2, Q, NB, CL, GRID>(pl, a, grid, st);
+        case 3: return launch_tc_t<3, Q, NB, CL, GRID>(pl, a, grid, st);
+        case 4: return launch_tc_t<4, Q, NB, CL, GRID>(pl, a, grid, st);
+        case 5: return launch_tc_t<5, Q, NB, CL, GRID>(pl, a, grid, st);
+        case 6: return launch_tc_t<6, Q, NB, CL, GRID>(pl, a, grid, st);
+        case 7: return launch_tc_t<7, Q, NB, CL, GRID>(pl, a, grid, st);
+        case 8: return launch_tc_t<8, Q, NB, CL, GRID>(pl, a, grid, st);
         default: return cudaErrorInvalidValue;
     }
+}
+
+template <bool GRID>
+cudaError_t launch_tc(int m, int v, const TcPlan& pl, const tc::TcArgs& a, int grid, cudaStream_t st)
+{
+    return v == 1 ? launch_tc_v<1, GRID>(m, pl, a, grid, st) : launch_tc_v<2, GRID>(m, pl, a, grid, st);
+}
+
+// Regions for the CTA-pair variant: an even number that divides the tiles (equal tile counts per pair).
+int choose_regions_pair(const dock_ctx* ctx, int64_t n_blocks, int nt)
+{
+    int best = 0;
+    double best_cost = 1e300;
+    for (int G = 2; G <= std::min(nt, 1024); G += 2) {
+        if (nt % G) continue;
+        if (ctx->regions_override > 0 && G != ctx->regions_override) continue;
+        const int tpr = nt / G;
+        const int64_t items = n_blocks * G;
+        const int64_t waves = (items + ctx->n_sms - 1) / ctx->n_sms;
+        const double cost = double(waves) * (tpr + 0.5);
+        if (cost < best_cost - 1e-9) {
+            best_cost = cost;
+            best = G;
+        }
+    }
+    return best;
 }
 
 // Regions per item for a given number of rotation batches and tiles.
@@ -592,21 +638,21 @@ dock_status run_fallback(dock_ctx* ctx, int m, int nfb, int64_t unit_begin, int 
     return DOCK_OK;
 }
 
-tc::TcArgs tc_args(dock_ctx* ctx, int m, int n_slots, int G, const unsigned char* W)
+tc::TcArgs tc_args(dock_ctx* ctx, int m, int v, int n_slots, int G, const unsigned char* W)
 {
-    const TcPlan& tp = ctx->tcplan[m];
+    const TcPlan& tp = ctx->tcplan[v][m];
     tc::TcArgs a{};
     a.nx = ctx->nx;
     a.ny = ctx->ny;
     a.nz = ctx->nz;
     a.ntx = ctx->tc_ntx;
-    a.nty = ctx->tc_nty;
+    a.nty = tc_nty(ctx, v);
     a.ntz = ctx->tc_ntz;
-    a.ntiles = ctx->tc_ntiles;
+    a.ntiles = tc_ntiles(ctx, v);
     a.G_ch = ctx->tc_Gch;
     a.n_slots = n_slots;
     a.G = G;
-    a.tiles_per_region = (ctx->tc_ntiles + G - 1) / G;
+    a.tiles_per_region = (a.ntiles + G - 1) / G;
     a.nsteps = tp.nsteps;
     a.W = W;
     a.TXB = tp.TXB;
@@ -619,20 +665,43 @@ tc::TcArgs tc_args(dock_ctx* ctx, int m, int n_slots, int G, const unsigned char
     return a;
 }
 
-// Engine choice: tensor cores when the plan for this m exists (auto) or when forced.
+// Variant + regions for a launch over n_slots rotations; returns false if the tensor cores can't run m.
+bool plan_tc_launch(dock_ctx* ctx, int m, int n_slots, int* v_out, int* G_out)
+{
+    const int64_t n_blocks = (n_slots + tc::ROT - 1) / tc::ROT;
+    const bool ok2 = ctx->tcplan[2][m].ok, ok1 = ctx->tcplan[1][m].ok;
+    if ((ctx->tc_variant == 0 || ctx->tc_variant == 2) && ok2) {
+        const int G = choose_regions_pair(ctx, n_blocks, tc_ntiles(ctx, 2));
+        if (G > 0) {
+            *v_out = 2;
+            *G_out = G;
+            return true;
+        }
+    }
+    if ((ctx->tc_variant == 0 || ctx->tc_variant == 1) && ok1) {
+        *v_out = 1;
+        *G_out = choose_regions_n(ctx, n_blocks, tc_ntiles(ctx, 1));
+        return true;
+    }
+    return false;
+}
+
+// Engine choice: tensor cores when a plan for this m exists (auto) or when forced.
 dock_status select_engine(dock_ctx* ctx, int m, bool* use_tc)
 {
-    const bool ok = ctx->tcplan[m].ok && (ctx->tc_q == 4 || m == 4);
+    int v = 0, G = 0;
+    const bool ok = plan_tc_launch(ctx, m, tc::ROT, &v, &G);
     if (ctx->engine == 2 && !ok) return fail(ctx, DOCK_E_UNSUPPORTED, "tensor-core engine unavailable for m=%d", m);
     *use_tc = ctx->engine == 2 || (ctx->engine == 0 && ok);
     ctx->engine_last = *use_tc ? 2 : 1;
+    if (!*use_tc) ctx->tc_variant_last = 0;
     return DOCK_OK;
 }
 
 // Pack folded FP32 weights into the tcgen05 A-operand layout.
 dock_status pack_weights_tc(dock_ctx* ctx, int m, int n_slots, const float* Lw)
 {
-    const TcPlan& tp = ctx->tcplan[m];
+    const TcPlan& tp = ctx->tcplan[1][m].ok ? ctx->tcplan[1][m] : ctx->tcplan[2][m];   // nsteps is variant-free
     const int64_t n_blocks = (n_slots + tc::ROT - 1) / tc::ROT;
     TRY(ensure(ctx, ctx->Wtc, (size_t)n_blocks * tp.nsteps * tc::WCHUNK));
     const int64_t rows = n_blocks * tp.nsteps * 2 * tc::ROT;
@@ -649,10 +718,11 @@ dock_status run_grid_tc(dock_ctx* ctx, int m, int n_slots, const float* Lw, floa
 {
     TRY(pack_weights_tc(ctx, m, n_slots, Lw));
     const int64_t n_blocks = (n_slots + tc::ROT - 1) / tc::ROT;
-    const int G = choose_regions_n(ctx, n_blocks, ctx->tc_ntiles);
-    tc::TcArgs a = tc_args(ctx, m, n_slots, G, static_cast<const unsigned char*>(ctx->Wtc.p));
+    int v = 0, G = 0;
+    if (!plan_tc_launch(ctx, m, n_slots, &v, &G)) return fail(ctx, DOCK_E_UNSUPPORTED, "no tensor-core plan");
+    tc::TcArgs a = tc_args(ctx, m, v, n_slots, G, static_cast<const unsigned char*>(ctx->Wtc.p));
     a.grid = grid;
-    CU(launch_tc<true>(m, ctx->tc_q, ctx->tcplan[m], a, (int)(n_blocks * G), ctx->stream));
+    CU(launch_tc<true>(m, v, ctx->tcplan[v][m], a, (int)(n_blocks * G), ctx->stream));
     ctx->kernels_last++;
     return DOCK_OK;
 }
@@ -803,15 +873,11 @@ dock_status dock_init(const dock_grid_desc* g, const float* receptor, const floa
                                                        G.Zp, P);
     // tcgen05 engine: bf16-split, channel-grouped, cyclic-halo copy of the receptor
     {
-        const char* q_env = getenv("DOCK_TC_Q");
-        if (q_env && atoi(q_env) == 2) ctx->tc_q = 2;
         ctx->tc_Gch = (P + 3) / 4;
         ctx->tc_ntx = (ctx->nx + tc::NT - 1) / tc::NT;
-        ctx->tc_nty = (ctx->ny + ctx->tc_q - 1) / ctx->tc_q;
         ctx->tc_ntz = ctx->nz;
-        ctx->tc_ntiles = ctx->tc_ntx * ctx->tc_nty * ctx->tc_ntz;
         ctx->tc_Xp = round_up((ctx->tc_ntx - 1) * tc::NT + tc_txb(ctx->m_max), 2);
-        ctx->tc_Yp = ctx->tc_nty * ctx->tc_q + ctx->m_max - 1;
+        ctx->tc_Yp = round_up(ctx->ny, 4) + ctx->m_max - 1;   // covers Q = 4 and Q = 2 tilings
         ctx->tc_Zp = ctx->nz + ctx->m_max - 1;
         const size_t bytes = (size_t)ctx->tc_Gch * ctx->tc_Zp * ctx->tc_Yp * ctx->tc_Xp * 16;
         if (cudaMalloc(&ctx->d_rec_tc, bytes) == cudaSuccess) {
@@ -831,7 +897,7 @@ dock_status dock_init(const dock_grid_desc* g, const float* receptor, const floa
     for (int m = 1; m <= ctx->m_max; m++) {
         dock_status s = make_plan(ctx, m);
         if (s != DOCK_OK && m == ctx->m_max) return bail(s);
-        if (make_tc_plan(ctx, m) != DOCK_OK) return bail(DOCK_E_CUDA);
+        if (make_tc_plan(ctx, m, 1) != DOCK_OK || make_tc_plan(ctx, m, 2) != DOCK_OK) return bail(DOCK_E_CUDA);
     }
     *out = ctx;
     return DOCK_OK;
@@ -849,6 +915,10 @@ dock_status dock_set_tuning(dock_ctx* ctx, int key, int64_t value)
         case DOCK_TUNE_ENGINE:
             if (value < 0 || value > 2) return fail(ctx, DOCK_E_INVALID_ARG, "engine must be 0 (auto), 1 (FFMA) or 2 (tcgen05)");
             ctx->engine = (int)value;
+            return DOCK_OK;
+        case DOCK_TUNE_TC_VARIANT:
+            if (value < 0 || value > 2) return fail(ctx, DOCK_E_INVALID_ARG, "tc variant must be 0, 1 or 2");
+            ctx->tc_variant = (int)value;
             return DOCK_OK;
         case DOCK_TUNE_CAND_CAP:
             if (value < 32 || value > (1 << 20)) return fail(ctx, DOCK_E_INVALID_ARG, "cand cap out of range");
@@ -889,7 +959,8 @@ dock_status dock_get_info(const dock_ctx* ctx, dock_info* info)
     }
     info->n_sms = ctx->n_sms;
     info->engine_last = ctx->engine_last;
-    info->tc_available = ctx->tcplan[ctx->m_max].ok ? 1 : 0;
+    info->tc_available = (ctx->tcplan[1][ctx->m_max].ok || ctx->tcplan[2][ctx->m_max].ok) ? 1 : 0;
+    info->tc_variant_last = ctx->tc_variant_last;
     return DOCK_OK;
 }
 
@@ -966,8 +1037,10 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
     if (use_tc) {
         TRY(pack_weights_tc(ctx, m, n_units, static_cast<const float*>(ctx->Lw.p)));
         const int64_t n_blocks = (n_units + tc::ROT - 1) / tc::ROT;
-        const int G = choose_regions_n(ctx, n_blocks, ctx->tc_ntiles);
-        tc::TcArgs ta = tc_args(ctx, m, n_units, G, static_cast<const unsigned char*>(ctx->Wtc.p));
+        int v = 0, G = 0;
+        if (!plan_tc_launch(ctx, m, n_units, &v, &G)) return fail(ctx, DOCK_E_UNSUPPORTED, "no tensor-core plan");
+        ctx->tc_variant_last = v;
+        tc::TcArgs ta = tc_args(ctx, m, v, n_units, G, static_cast<const unsigned char*>(ctx->Wtc.p));
         ta.k = k;
         ta.rho = rho;
         ta.cap = cap;
@@ -978,7 +1051,7 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
         const int64_t items = n_blocks * G;
         if (items > 0x7fffffff) return fail(ctx, DOCK_E_UNSUPPORTED, "too many work items");
         CU(cudaEventRecord(ctx->ev_corr[0], ctx->stream));
-        CU(launch_tc<false>(m, ctx->tc_q, ctx->tcplan[m], ta, (int)items, ctx->stream));
+        CU(launch_tc<false>(m, v, ctx->tcplan[v][m], ta, (int)items, ctx->stream));
         CU(cudaEventRecord(ctx->ev_corr[1], ctx->stream));
         ctx->regions_last = G;
         ctx->items_last = items;

@@ -151,7 +151,34 @@ __device__ __forceinline__ void list_insert(unsigned long long (&L)[LIST], unsig
     L[0] = key < L[0] ? key : L[0];
 }
 
-template <int M, int Q, int NBUF, bool GRID>
+__device__ __forceinline__ void cluster_sync_all()
+{
+    asm volatile("barrier.cluster.arrive.release.aligned;\n\tbarrier.cluster.wait.acquire.aligned;" ::: "memory");
+}
+// Bulk copy global -> the same shared offset in every CTA of ctaMask, completing tx on each CTA's barrier.
+__device__ __forceinline__ void bulk_load_mc(void* dst, const void* src, unsigned bytes, uint64_t* bar, uint16_t mask)
+{
+    asm volatile(
+        "cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes.multicast::cluster [%0], [%1], %2, [%3], %4;" ::"r"(
+            dk::smem_u32(dst)),
+        "l"(src), "r"(bytes), "r"(dk::smem_u32(bar)), "h"(mask)
+        : "memory");
+}
+__device__ __forceinline__ void umma_commit_mc(uint64_t* bar, uint16_t mask)
+{
+    asm volatile(
+        "tcgen05.commit.cta_group::1.mbarrier::arrive::one.shared::cluster.multicast::cluster.b64 [%0], %1;" ::"r"(
+            dk::smem_u32(bar)),
+        "h"(mask)
+        : "memory");
+}
+
+// CL = 1: one CTA per item.  CL = 2: a cluster of two CTAs works on the same rotation block
+// (two regions with the same number of tiles); each CTA's producer fetches half of every
+// weight chunk and multicasts it into both CTAs' rings, and each MMA warp releases a ring
+// slot in both CTAs -- the weight stream from L2 is halved, which lets Q = 2 rows per TMEM
+// buffer with NBUF = 2 buffers (epilogue overlapped with the next tile's MMAs).
+template <int M, int Q, int NBUF, int CL, bool GRID>
 __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__ CUtensorMap tmap, const TcArgs a)
 {
     static_assert(Q * NBUF * NT <= 512, "TMEM has 512 columns");
@@ -181,7 +208,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
         }
         for (int i = 0; i < a.wstages; i++) {
             dk::mbar_init(&w_full[i], 1);
-            dk::mbar_init(&w_empty[i], 1);
+            dk::mbar_init(&w_empty[i], CL);
         }
         for (int i = 0; i < NBUF; i++) {
             dk::mbar_init(&tm_full[i], 1);
@@ -196,8 +223,12 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
     }
     tc_fence_before();
     __syncthreads();
+    if constexpr (CL > 1) cluster_sync_all();   // peers' barriers are initialised before any multicast
     tc_fence_after();
     const uint32_t tmem = tmem_base_s;
+    uint32_t crank = 0;
+    if constexpr (CL > 1) asm volatile("mov.u32 %0, %%cluster_ctarank;" : "=r"(crank));
+    constexpr uint16_t CMASK = (1u << CL) - 1u;
 
     if (n_tiles > 0) {
         if (warp == 0) {
@@ -223,11 +254,28 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                     if (wuse >= a.wstages) dk::mbar_wait(&w_empty[ws], wph ^ 1);
                     if (elect_one()) {
                         dk::mbar_arrive_expect_tx(&w_full[ws], WCHUNK);
-                        dk::bulk_load(w_smem + static_cast<size_t>(ws) * WCHUNK, wsrc + static_cast<size_t>(s) * WCHUNK,
-                                      WCHUNK, &w_full[ws]);
+                        if constexpr (CL == 1) {
+                            dk::bulk_load(w_smem + static_cast<size_t>(ws) * WCHUNK,
+                                          wsrc + static_cast<size_t>(s) * WCHUNK, WCHUNK, &w_full[ws]);
+                        } else {
+                            constexpr unsigned HALF = WCHUNK / CL;
+                            bulk_load_mc(w_smem + static_cast<size_t>(ws) * WCHUNK + crank * HALF,
+                                         wsrc + static_cast<size_t>(s) * WCHUNK + crank * HALF, HALF, &w_full[ws],
+                                         CMASK);
+                        }
                     }
                     __syncwarp();
                     wuse++;
+                    if (++ws == a.wstages) {
+                        ws = 0;
+                        wph ^= 1;
+                    }
+                }
+            }
+            if constexpr (CL > 1) {
+                // drain: every ring slot's last release (from both MMA warps) has arrived before exit
+                for (int i = 0; i < min(wuse, a.wstages); i++) {
+                    dk::mbar_wait(&w_empty[ws], wph ^ 1);
                     if (++ws == a.wstages) {
                         ws = 0;
                         wph ^= 1;
@@ -266,7 +314,8 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
 #pragma unroll
                                         for (int q = 0; q < Q; q++)
                                             umma_bf16(dcol + q * NT, da, db + ((q * row16) >> 4), idesc, acc);
-                                        umma_commit(&w_empty[ws]);
+                                        if constexpr (CL == 1) umma_commit(&w_empty[ws]);
+                                        else umma_commit_mc(&w_empty[ws], CMASK);
                                     }
                                     __syncwarp();
                                     acc = 1;
@@ -392,6 +441,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
     tc_fence_before();
     __syncthreads();
     if (warp == 1) asm volatile("tcgen05.dealloc.cta_group::1.sync.aligned.b32 %0, 512;" ::"r"(tmem));
+    if constexpr (CL > 1) cluster_sync_all();
 }
 
 // ------------------------------------------------------------------ data preparation

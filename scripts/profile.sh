@@ -7,11 +7,12 @@ set -u
 mkdir -p gpurun_out
 TAG=${1:-r01}
 ENGINE=${2:-auto}
+KRE=k_corr; [ "$ENGINE" = "tc" ] && KRE=k_corr_tc
 CMD="python bench.py --steps 2 --warmup 1 --no-e2e --no-cpu-baseline --no-alt --engine $ENGINE"
 timeout 900 ncu --metrics gpu__time_duration.sum --clock-control none --csv \
     --log-file gpurun_out/launches_${TAG}_${ENGINE}.csv $CMD > gpurun_out/launches_${TAG}_${ENGINE}.log 2>&1
 echo "launch list rc=$?"
-timeout 1500 ncu --set full --clock-control none --import-source on -k regex:k_corr -s 1 -c 1 \
+timeout 1500 ncu --set full --clock-control none --import-source on -k regex:$KRE -s 1 -c 1 \
     -o gpurun_out/corr_${TAG}_${ENGINE} -f $CMD > gpurun_out/corr_${TAG}_${ENGINE}.log 2>&1
 echo "full capture rc=$?"
 ncu -i gpurun_out/corr_${TAG}_${ENGINE}.ncu-rep --page raw --csv > gpurun_out/corr_${TAG}_${ENGINE}_raw.csv 2>/dev/null

@@ -26,14 +26,22 @@ def D():
     return D
 
 
-ENGINES = [1, 2]          # DOCK_TUNE_ENGINE: 1 = FP32 FFMA, 2 = tcgen05 bf16x3
+# engine ids used by the tests: 1 = FP32 FFMA; 2 = tcgen05 variant 1 (4 rows, 1 TMEM buffer);
+# 3 = tcgen05 variant 2 (2 rows, 2 TMEM buffers, CTA pair with multicast weights)
+ENGINES = [1, 2, 3]
 
 
 def _ctx(D, R, w, m_max, engine=0):
     ctx = D.dock_init(R, w, H, m_max=m_max)
     if engine:
-        D.dock_set_tuning(ctx, D.DOCK_TUNE_ENGINE, engine)
+        D.dock_set_tuning(ctx, D.DOCK_TUNE_ENGINE, 1 if engine == 1 else 2)
+        if engine >= 2:
+            D.dock_set_tuning(ctx, D.DOCK_TUNE_TC_VARIANT, engine - 1)
     return ctx
+
+
+def _engine_id(info):
+    return 1 if info["engine_last"] == 1 else 1 + info["tc_variant_last"]
 
 
 def _oracle_SA(orc, R, w, pr, q):
@@ -180,7 +188,7 @@ def test_poses_mid_config(D, orc, kind, rho, engine):
     probes = g.probes(3, m, P)
     rot = g.rotations(21)
     _, info, mism = _dock_and_validate(D, orc, R, w, probes, rot, 4, rho, engine=engine)
-    assert info["engine_last"] == engine
+    assert _engine_id(info) == engine
     assert info["fallback_last"] <= 2
 
 
@@ -329,7 +337,7 @@ def test_prod_config_sampled(D, orc, engine):
     rot = g.rotations(c.n_rot)
     units = [0, 1, 499, 500, 3777, 7999] + list(range(137, 8000, 811))
     _, info, _ = _dock_and_validate(D, orc, R, w, probes, rot, c.k, 1, units=units, engine=engine)
-    assert info["fallback_last"] <= 80 and info["engine_last"] == engine
+    assert info["fallback_last"] <= 80 and _engine_id(info) == engine
 
 
 def test_large_config_sampled(D, orc):
