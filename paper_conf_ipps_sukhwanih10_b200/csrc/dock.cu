@@ -285,12 +285,13 @@ dock_status make_tc_plan(dock_ctx* ctx, int m, int v)
     pl.rec_stage_bytes = round_up(ctx->tc_Gch * pl.box_bytes, 1024);
     pl.nsteps = ctx->tc_Gch * 2 * m * m * ((m + 1) / 2);
     const int budget = kSmemLimit - 2048;   // static shared memory (barriers) and slack
-    const int min_ring = 4 * tc::WCHUNK;
+    const int stage = tc::KSTEPS * tc::WCHUNK;
+    const int min_ring = 3 * stage;
     if (2 * pl.rec_stage_bytes + min_ring <= budget) pl.n_rec_stages = 2;
     else if (pl.rec_stage_bytes + min_ring <= budget) pl.n_rec_stages = 1;
     else return DOCK_OK;                    // this m is not eligible for the tensor-core engine
-    pl.wstages = std::min(tc::WSTAGES, (budget - pl.n_rec_stages * pl.rec_stage_bytes) / tc::WCHUNK);
-    const int ring = pl.wstages * tc::WCHUNK;
+    pl.wstages = std::min(tc::WSTAGES, (budget - pl.n_rec_stages * pl.rec_stage_bytes) / stage);
+    const int ring = pl.wstages * stage;
     // >= 116 KB keeps one CTA per SM: every CTA allocates all 512 TMEM columns
     pl.smem = std::max(pl.n_rec_stages * pl.rec_stage_bytes + ring, 116 * 1024);
     auto fn = encode_fn();
@@ -670,7 +671,8 @@ bool plan_tc_launch(dock_ctx* ctx, int m, int n_slots, int* v_out, int* G_out)
 {
     const int64_t n_blocks = (n_slots + tc::ROT - 1) / tc::ROT;
     const bool ok2 = ctx->tcplan[2][m].ok, ok1 = ctx->tcplan[1][m].ok;
-    if ((ctx->tc_variant == 0 || ctx->tc_variant == 2) && ok2) {
+    // the variant setting is a preference: variant 2 needs an even region count dividing the tiles
+    if (ctx->tc_variant != 1 && ok2) {
         const int G = choose_regions_pair(ctx, n_blocks, tc_ntiles(ctx, 2));
         if (G > 0) {
             *v_out = 2;
@@ -678,7 +680,7 @@ bool plan_tc_launch(dock_ctx* ctx, int m, int n_slots, int* v_out, int* G_out)
             return true;
         }
     }
-    if ((ctx->tc_variant == 0 || ctx->tc_variant == 1) && ok1) {
+    if (ok1) {
         *v_out = 1;
         *G_out = choose_regions_n(ctx, n_blocks, tc_ntiles(ctx, 1));
         return true;

@@ -33,6 +33,7 @@ constexpr int NEPI = 8;         // epilogue warps (2 per TMEM lane quarter)
 constexpr int NTHREADS = (2 + NEPI) * 32;
 constexpr int WSTAGES = 16;     // max weight ring depth (runtime a.wstages <= 16; 16 x 4 KB covers the L2 latency)
 constexpr int WCHUNK = 2 * ROT * 16;   // bytes of one K-step of A (2 K-chunks x 128 rotations x 16 B)
+constexpr int KSTEPS = 2;       // K-steps of A per ring stage (nsteps is always even: 2 passes)
 constexpr int LIST = 32;        // per-thread candidate list (exact top-LIST keys of one rotation)
 
 struct TcArgs {
@@ -181,6 +182,8 @@ __device__ __forceinline__ void umma_commit_mc(uint64_t* bar, uint16_t mask)
 template <int M, int Q, int NBUF, int CL, bool GRID>
 __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__ CUtensorMap tmap, const TcArgs a)
 {
+    constexpr int KS = KSTEPS;                 // K-steps per weight-ring stage (one wait/commit per KS steps)
+    constexpr unsigned STAGE = KS * WCHUNK;
     static_assert(Q * NBUF * NT <= 512, "TMEM has 512 columns");
     constexpr int MXP = (M + 1) / 2;   // voxel pairs along x (K = 16 = 2 voxels x 8 channels)
     extern __shared__ __align__(1024) unsigned char smem[];
@@ -250,16 +253,16 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                                     &rec_full[rs]);
                 }
                 __syncwarp();
-                for (int s = 0; s < a.nsteps; s++) {
+                for (int s = 0; s < a.nsteps; s += KS) {
                     if (wuse >= a.wstages) dk::mbar_wait(&w_empty[ws], wph ^ 1);
                     if (elect_one()) {
-                        dk::mbar_arrive_expect_tx(&w_full[ws], WCHUNK);
+                        dk::mbar_arrive_expect_tx(&w_full[ws], STAGE);
                         if constexpr (CL == 1) {
-                            dk::bulk_load(w_smem + static_cast<size_t>(ws) * WCHUNK,
-                                          wsrc + static_cast<size_t>(s) * WCHUNK, WCHUNK, &w_full[ws]);
+                            dk::bulk_load(w_smem + static_cast<size_t>(ws) * STAGE,
+                                          wsrc + static_cast<size_t>(s) * WCHUNK, STAGE, &w_full[ws]);
                         } else {
-                            constexpr unsigned HALF = WCHUNK / CL;
-                            bulk_load_mc(w_smem + static_cast<size_t>(ws) * WCHUNK + crank * HALF,
+                            constexpr unsigned HALF = STAGE / CL;
+                            bulk_load_mc(w_smem + static_cast<size_t>(ws) * STAGE + crank * HALF,
                                          wsrc + static_cast<size_t>(s) * WCHUNK + crank * HALF, HALF, &w_full[ws],
                                          CMASK);
                         }
@@ -289,7 +292,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
             const uint64_t dA0 = umma_desc(w0, ROT * 16, 128);   // + (slot offset >> 4)
             const uint64_t dB0 = umma_desc(rec0, 16, 128);       // + (voxel offset >> 4)
             const uint32_t row16 = static_cast<uint32_t>(a.TXB) * 16u;
-            int ws = 0, wph = 0;
+            int ws = 0, wph = 0, kin = 0;
             for (int ti = 0; ti < n_tiles; ti++) {
                 const int rs = ti % a.n_rec_stages, ruse = ti / a.n_rec_stages;
                 const int buf = ti % NBUF, buse = ti / NBUF;
@@ -306,22 +309,30 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                                 const uint32_t rowofs = gofs + static_cast<uint32_t>(vz * a.TYB + vy) * row16;
 #pragma unroll
                                 for (int vxp = 0; vxp < MXP; vxp++) {
-                                    dk::mbar_wait(&w_full[ws], wph);
-                                    tc_fence_after();
+                                    if (kin == 0) {
+                                        dk::mbar_wait(&w_full[ws], wph);
+                                        tc_fence_after();
+                                    }
                                     if (elect_one()) {
-                                        const uint64_t da = dA0 + ((static_cast<uint32_t>(ws) * WCHUNK) >> 4);
+                                        const uint64_t da =
+                                            dA0 + ((static_cast<uint32_t>(ws) * STAGE + kin * WCHUNK) >> 4);
                                         const uint64_t db = dB0 + ((rowofs + vxp * 32u) >> 4);
 #pragma unroll
                                         for (int q = 0; q < Q; q++)
                                             umma_bf16(dcol + q * NT, da, db + ((q * row16) >> 4), idesc, acc);
-                                        if constexpr (CL == 1) umma_commit(&w_empty[ws]);
-                                        else umma_commit_mc(&w_empty[ws], CMASK);
+                                        if (kin == KS - 1) {
+                                            if constexpr (CL == 1) umma_commit(&w_empty[ws]);
+                                            else umma_commit_mc(&w_empty[ws], CMASK);
+                                        }
                                     }
                                     __syncwarp();
                                     acc = 1;
-                                    if (++ws == a.wstages) {
-                                        ws = 0;
-                                        wph ^= 1;
+                                    if (++kin == KS) {
+                                        kin = 0;
+                                        if (++ws == a.wstages) {
+                                            ws = 0;
+                                            wph ^= 1;
+                                        }
                                     }
                                 }
                             }
