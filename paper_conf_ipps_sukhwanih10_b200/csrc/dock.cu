@@ -34,7 +34,9 @@ struct DevBuf {
 
 struct TcPlan {                // per-probe-size plan of the tcgen05 engine
     bool ok = false;
-    CUtensorMap tmap;
+    bool pair = false;         // PAIR scheme (one channel group): second receptor copy (Rhi(x), Rhi(x+1))
+    CUtensorMap tmap, tmap_pair;
+    int S1 = 0, S1p = 0, S2 = 0, S2p = 0;
     int TXB = 0, TYB = 0, TZB = 0, box_bytes = 0, rec_stage_bytes = 0, n_rec_stages = 0, smem = 0, nsteps = 0,
         wstages = 0;
 };
@@ -68,6 +70,7 @@ struct dock_ctx {
     int tc_variant = 0;        // DOCK_TUNE_TC_VARIANT: 0 auto, 1 (Q4, 1 TMEM buffer), 2 (Q2, 2 buffers, CTA pair)
     int tc_variant_last = 0;
     uint16_t* d_rec_tc = nullptr;
+    uint16_t* d_rec_pair = nullptr;   // PAIR-scheme receptor copy (P <= 4)
     int tc_Gch = 0, tc_ntx = 0, tc_ntz = 0, tc_Xp = 0, tc_Yp = 0, tc_Zp = 0;
     TcPlan tcplan[3][DOCK_MAX_M + 1];   // [variant][m]
     DevBuf Wtc;
@@ -274,21 +277,34 @@ inline int tc_cl(int v) { return v == 1 ? 1 : 2; }
 inline int tc_nty(const dock_ctx* c, int v) { return (c->ny + tc_q(v) - 1) / tc_q(v); }
 inline int tc_ntiles(const dock_ctx* c, int v) { return c->tc_ntx * tc_nty(c, v) * c->tc_ntz; }
 
+int tc_txb_any(int m) { return std::max(tc_txb(m), 4 * ((m + 3) / 4) + 126); }
+
 dock_status make_tc_plan(dock_ctx* ctx, int m, int v)
 {
     TcPlan& pl = ctx->tcplan[v][m];
     if (pl.ok || !ctx->d_rec_tc) return DOCK_OK;
-    pl.TXB = tc_txb(m);
+    pl.pair = ctx->tc_Gch == 1 && ctx->d_rec_pair != nullptr;
+    if (!pl.pair && v != 1) return DOCK_OK;          // the CTA-pair variant is built for the PAIR scheme only
+    const int KS = tc::KSTEPS;
+    pl.TXB = pl.pair ? tc_txb_any(m) : tc_txb(m);
     pl.TYB = tc_q(v) + m - 1;
     pl.TZB = m;
     pl.box_bytes = 16 * pl.TXB * pl.TYB * pl.TZB;
     pl.rec_stage_bytes = round_up(ctx->tc_Gch * pl.box_bytes, 1024);
-    pl.nsteps = ctx->tc_Gch * 2 * m * m * ((m + 1) / 2);
+    if (pl.pair) {
+        pl.S1 = m * m * ((m + 1) / 2);
+        pl.S1p = round_up(pl.S1, KS);
+        pl.S2 = m * m * ((m + 3) / 4);
+        pl.S2p = round_up(pl.S2, KS);
+        pl.nsteps = pl.S1p + pl.S2p;
+    } else {
+        pl.nsteps = ctx->tc_Gch * 2 * m * m * ((m + 1) / 2);
+    }
     const int budget = kSmemLimit - 2048;   // static shared memory (barriers) and slack
-    const int stage = tc::KSTEPS * tc::WCHUNK;
+    const int stage = KS * tc::WCHUNK;
     const int min_ring = 3 * stage;
     if (2 * pl.rec_stage_bytes + min_ring <= budget) pl.n_rec_stages = 2;
-    else if (pl.rec_stage_bytes + min_ring <= budget) pl.n_rec_stages = 1;
+    else if (!pl.pair && pl.rec_stage_bytes + min_ring <= budget) pl.n_rec_stages = 1;
     else return DOCK_OK;                    // this m is not eligible for the tensor-core engine
     pl.wstages = std::min(tc::WSTAGES, (budget - pl.n_rec_stages * pl.rec_stage_bytes) / stage);
     const int ring = pl.wstages * stage;
@@ -301,22 +317,26 @@ dock_status make_tc_plan(dock_ctx* ctx, int m, int v)
     cuuint64_t strides[4] = {16, X * 16, X * Y * 16, X * Y * Z * 16};
     cuuint32_t box[5] = {8, (cuuint32_t)pl.TXB, (cuuint32_t)pl.TYB, (cuuint32_t)pl.TZB, 1};
     cuuint32_t es[5] = {1, 1, 1, 1, 1};
-    CUresult r = fn(&pl.tmap, CU_TENSOR_MAP_DATA_TYPE_BFLOAT16, 5, ctx->d_rec_tc, dims, strides, box, es,
-                    CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_L2_256B,
-                    CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
-    if (r != CUDA_SUCCESS) return fail(ctx, DOCK_E_CUDA, "cuTensorMapEncodeTiled (bf16) failed (%d)", (int)r);
+    for (int which = 0; which < (pl.pair ? 2 : 1); which++) {
+        CUresult r = fn(which ? &pl.tmap_pair : &pl.tmap, CU_TENSOR_MAP_DATA_TYPE_BFLOAT16, 5,
+                        which ? (void*)ctx->d_rec_pair : (void*)ctx->d_rec_tc, dims, strides, box, es,
+                        CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_L2_256B,
+                        CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+        if (r != CUDA_SUCCESS) return fail(ctx, DOCK_E_CUDA, "cuTensorMapEncodeTiled (bf16) failed (%d)", (int)r);
+    }
+    if (!pl.pair) pl.tmap_pair = pl.tmap;
     pl.ok = true;
     return DOCK_OK;
 }
 
-template <int M, int Q, int NBUF, int CL, bool GRID>
+template <int M, int Q, int NBUF, int CL, bool PAIR, bool GRID>
 cudaError_t launch_tc_t(const TcPlan& pl, const tc::TcArgs& a, int grid, cudaStream_t st)
 {
-    auto kern = tc::k_corr_tc<M, Q, NBUF, CL, GRID>;
+    auto kern = tc::k_corr_tc<M, Q, NBUF, CL, PAIR, GRID>;
     cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, pl.smem);
     if (e != cudaSuccess) return e;
     if constexpr (CL == 1) {
-        kern<<<grid, tc::NTHREADS, pl.smem, st>>>(pl.tmap, a);
+        kern<<<grid, tc::NTHREADS, pl.smem, st>>>(pl.tmap, pl.tmap_pair, a);
     } else {
         cudaLaunchConfig_t cfg{};
         cfg.gridDim = dim3(grid);
@@ -330,25 +350,25 @@ cudaError_t launch_tc_t(const TcPlan& pl, const tc::TcArgs& a, int grid, cudaStr
         at[0].val.clusterDim.z = 1;
         cfg.attrs = at;
         cfg.numAttrs = 1;
-        e = cudaLaunchKernelEx(&cfg, kern, pl.tmap, a);
+        e = cudaLaunchKernelEx(&cfg, kern, pl.tmap, pl.tmap_pair, a);
         if (e != cudaSuccess) return e;
     }
     return cudaGetLastError();
 }
 
-template <int V, bool GRID>
+template <int V, bool PAIR, bool GRID>
 cudaError_t launch_tc_v(int m, const TcPlan& pl, const tc::TcArgs& a, int grid, cudaStream_t st)
 {
     constexpr int Q = V == 1 ? 4 : 2, NB = V == 1 ? 1 : 2, CL = V == 1 ? 1 : 2;
     switch (m) {
-        case 1: return launch_tc_t<1, Q, NB, CL, GRID>(pl, a, grid, st);
-        case 2: return launch_tc_t<2, Q, NB, CL, GRID>(pl, a, grid, st);
-        case 3: return launch_tc_t<3, Q, NB, CL, GRID>(pl, a, grid, st);
-        case 4: return launch_tc_t<4, Q, NB, CL, GRID>(pl, a, grid, st);
-        case 5: return launch_tc_t<5, Q, NB, CL, GRID>(pl, a, grid, st);
-        case 6: return launch_tc_t<6, Q, NB, CL, GRID>(pl, a, grid, st);
-        case 7: return launch_tc_t<7, Q, NB, CL, GRID>(pl, a, grid, st);
-        case 8: return launch_tc_t<8, Q, NB, CL, GRID>(pl, a, grid, st);
+        case 1: return launch_tc_t<1, Q, NB, CL, PAIR, GRID>(pl, a, grid, st);
+        case 2: return launch_tc_t<2, Q, NB, CL, PAIR, GRID>(pl, a, grid, st);
+        case 3: return launch_tc_t<3, Q, NB, CL, PAIR, GRID>(pl, a, grid, st);
+        case 4: return launch_tc_t<4, Q, NB, CL, PAIR, GRID>(pl, a, grid, st);
+        case 5: return launch_tc_t<5, Q, NB, CL, PAIR, GRID>(pl, a, grid, st);
+        case 6: return launch_tc_t<6, Q, NB, CL, PAIR, GRID>(pl, a, grid, st);
+        case 7: return launch_tc_t<7, Q, NB, CL, PAIR, GRID>(pl, a, grid, st);
+        case 8: return launch_tc_t<8, Q, NB, CL, PAIR, GRID>(pl, a, grid, st);
         default: return cudaErrorInvalidValue;
     }
 }
@@ -356,7 +376,8 @@ cudaError_t launch_tc_v(int m, const TcPlan& pl, const tc::TcArgs& a, int grid, 
 template <bool GRID>
 cudaError_t launch_tc(int m, int v, const TcPlan& pl, const tc::TcArgs& a, int grid, cudaStream_t st)
 {
-    return v == 1 ? launch_tc_v<1, GRID>(m, pl, a, grid, st) : launch_tc_v<2, GRID>(m, pl, a, grid, st);
+    if (!pl.pair) return v == 1 ? launch_tc_v<1, false, GRID>(m, pl, a, grid, st) : cudaErrorInvalidValue;
+    return v == 1 ? launch_tc_v<1, true, GRID>(m, pl, a, grid, st) : launch_tc_v<2, true, GRID>(m, pl, a, grid, st);
 }
 
 // Regions for the CTA-pair variant: an even number that divides the tiles (equal tile counts per pair).
@@ -663,6 +684,10 @@ tc::TcArgs tc_args(dock_ctx* ctx, int m, int v, int n_slots, int G, const unsign
     a.rec_stage_bytes = tp.rec_stage_bytes;
     a.n_rec_stages = tp.n_rec_stages;
     a.wstages = tp.wstages;
+    a.S1 = tp.S1;
+    a.S1p = tp.S1p;
+    a.S2 = tp.S2;
+    a.S2p = tp.S2p;
     return a;
 }
 
@@ -671,8 +696,9 @@ bool plan_tc_launch(dock_ctx* ctx, int m, int n_slots, int* v_out, int* G_out)
 {
     const int64_t n_blocks = (n_slots + tc::ROT - 1) / tc::ROT;
     const bool ok2 = ctx->tcplan[2][m].ok, ok1 = ctx->tcplan[1][m].ok;
-    // the variant setting is a preference: variant 2 needs an even region count dividing the tiles
-    if (ctx->tc_variant != 1 && ok2) {
+    // variant 1 is the default (fastest measured); variant 2 only when asked for and possible
+    // (it needs an even region count dividing the tiles)
+    if (ctx->tc_variant == 2 && ok2) {
         const int G = choose_regions_pair(ctx, n_blocks, tc_ntiles(ctx, 2));
         if (G > 0) {
             *v_out = 2;
@@ -700,16 +726,19 @@ dock_status select_engine(dock_ctx* ctx, int m, bool* use_tc)
     return DOCK_OK;
 }
 
-// Pack folded FP32 weights into the tcgen05 A-operand layout.
-dock_status pack_weights_tc(dock_ctx* ctx, int m, int n_slots, const float* Lw)
+// Pack folded FP32 weights into the tcgen05 A-operand layout of plan tp.
+dock_status pack_weights_tc(dock_ctx* ctx, int m, const TcPlan& tp, int n_slots, const float* Lw)
 {
-    const TcPlan& tp = ctx->tcplan[1][m].ok ? ctx->tcplan[1][m] : ctx->tcplan[2][m];   // nsteps is variant-free
     const int64_t n_blocks = (n_slots + tc::ROT - 1) / tc::ROT;
     TRY(ensure(ctx, ctx->Wtc, (size_t)n_blocks * tp.nsteps * tc::WCHUNK));
     const int64_t rows = n_blocks * tp.nsteps * 2 * tc::ROT;
     const int grid = (int)std::min<int64_t>((rows + 255) / 256, 65535);
-    tc::k_pack_weights_tc<<<grid, 256, 0, ctx->stream>>>(Lw, static_cast<unsigned char*>(ctx->Wtc.p), n_slots, ctx->P,
-                                                          ctx->tc_Gch, m, tp.nsteps);
+    unsigned char* W = static_cast<unsigned char*>(ctx->Wtc.p);
+    if (tp.pair)
+        tc::k_pack_weights_tc_pair<<<grid, 256, 0, ctx->stream>>>(Lw, W, n_slots, ctx->P, m, tp.S1, tp.S1p, tp.S2,
+                                                                   tp.S2p);
+    else
+        tc::k_pack_weights_tc<<<grid, 256, 0, ctx->stream>>>(Lw, W, n_slots, ctx->P, ctx->tc_Gch, m, tp.nsteps);
     CU(cudaGetLastError());
     ctx->kernels_last++;
     return DOCK_OK;
@@ -718,10 +747,10 @@ dock_status pack_weights_tc(dock_ctx* ctx, int m, int n_slots, const float* Lw)
 // Score grids for n slots with the tensor-core engine (GRID epilogue).
 dock_status run_grid_tc(dock_ctx* ctx, int m, int n_slots, const float* Lw, float* grid)
 {
-    TRY(pack_weights_tc(ctx, m, n_slots, Lw));
     const int64_t n_blocks = (n_slots + tc::ROT - 1) / tc::ROT;
     int v = 0, G = 0;
     if (!plan_tc_launch(ctx, m, n_slots, &v, &G)) return fail(ctx, DOCK_E_UNSUPPORTED, "no tensor-core plan");
+    TRY(pack_weights_tc(ctx, m, ctx->tcplan[v][m], n_slots, Lw));
     tc::TcArgs a = tc_args(ctx, m, v, n_slots, G, static_cast<const unsigned char*>(ctx->Wtc.p));
     a.grid = grid;
     CU(launch_tc<true>(m, v, ctx->tcplan[v][m], a, (int)(n_blocks * G), ctx->stream));
@@ -762,6 +791,7 @@ void dock_destroy(dock_ctx* ctx)
         if (b->p) cudaFree(b->p);
     if (ctx->d_rec) cudaFree(ctx->d_rec);
     if (ctx->d_rec_tc) cudaFree(ctx->d_rec_tc);
+    if (ctx->d_rec_pair) cudaFree(ctx->d_rec_pair);
     if (ctx->Wtc.p) cudaFree(ctx->Wtc.p);
     if (ctx->d_w) cudaFree(ctx->d_w);
     if (ctx->d_eye) cudaFree(ctx->d_eye);
@@ -878,13 +908,25 @@ dock_status dock_init(const dock_grid_desc* g, const float* receptor, const floa
         ctx->tc_Gch = (P + 3) / 4;
         ctx->tc_ntx = (ctx->nx + tc::NT - 1) / tc::NT;
         ctx->tc_ntz = ctx->nz;
-        ctx->tc_Xp = round_up((ctx->tc_ntx - 1) * tc::NT + tc_txb(ctx->m_max), 2);
+        int txb_max = 0;
+        for (int mm = 1; mm <= ctx->m_max; mm++) txb_max = std::max(txb_max, tc_txb_any(mm));
+        ctx->tc_Xp = round_up((ctx->tc_ntx - 1) * tc::NT + txb_max, 2);
         ctx->tc_Yp = round_up(ctx->ny, 4) + ctx->m_max - 1;   // covers Q = 4 and Q = 2 tilings
         ctx->tc_Zp = ctx->nz + ctx->m_max - 1;
         const size_t bytes = (size_t)ctx->tc_Gch * ctx->tc_Zp * ctx->tc_Yp * ctx->tc_Xp * 16;
         if (cudaMalloc(&ctx->d_rec_tc, bytes) == cudaSuccess) {
             tc::k_pack_receptor_tc<<<2048, 256, 0, ctx->stream>>>(d_src, ctx->d_rec_tc, ctx->nx, ctx->ny, ctx->nz,
                                                                    ctx->tc_Xp, ctx->tc_Yp, ctx->tc_Zp, P, ctx->tc_Gch);
+            if (ctx->tc_Gch == 1) {
+                const size_t pbytes = (size_t)ctx->tc_Zp * ctx->tc_Yp * ctx->tc_Xp * 16;
+                if (cudaMalloc(&ctx->d_rec_pair, pbytes) == cudaSuccess) {
+                    tc::k_pack_receptor_pair_tc<<<2048, 256, 0, ctx->stream>>>(
+                        d_src, ctx->d_rec_pair, ctx->nx, ctx->ny, ctx->nz, ctx->tc_Xp, ctx->tc_Yp, ctx->tc_Zp, P);
+                } else {
+                    cudaGetLastError();
+                    ctx->d_rec_pair = nullptr;
+                }
+            }
         } else {
             cudaGetLastError();
             ctx->d_rec_tc = nullptr;   // the tensor-core engine is then unavailable
@@ -1037,10 +1079,10 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
     auto* cntp = static_cast<unsigned int*>(ctx->cnt.p);
     auto* candp = static_cast<unsigned long long*>(ctx->cand.p);
     if (use_tc) {
-        TRY(pack_weights_tc(ctx, m, n_units, static_cast<const float*>(ctx->Lw.p)));
         const int64_t n_blocks = (n_units + tc::ROT - 1) / tc::ROT;
         int v = 0, G = 0;
         if (!plan_tc_launch(ctx, m, n_units, &v, &G)) return fail(ctx, DOCK_E_UNSUPPORTED, "no tensor-core plan");
+        TRY(pack_weights_tc(ctx, m, ctx->tcplan[v][m], n_units, static_cast<const float*>(ctx->Lw.p)));
         ctx->tc_variant_last = v;
         tc::TcArgs ta = tc_args(ctx, m, v, n_units, G, static_cast<const unsigned char*>(ctx->Wtc.p));
         ta.k = k;

@@ -41,7 +41,8 @@ struct TcArgs {
     int ntx, nty, ntz, ntiles;  // tiles: 128 x Q rows (y) x 1 (z)
     int G_ch;                   // channel groups of 4
     int n_slots, G, tiles_per_region;
-    int nsteps;
+    int nsteps;                 // K-steps of A per tile (all passes, padded to multiples of KSTEPS)
+    int S1, S1p, S2, S2p;       // PAIR scheme: pass-1 steps (real, padded) and pass-2 steps (real, padded)
     const unsigned char* W;     // [block][step][WCHUNK]
     int TXB, TYB, TZB;
     int box_bytes;              // one channel group's receptor box
@@ -179,8 +180,12 @@ __device__ __forceinline__ void umma_commit_mc(uint64_t* bar, uint16_t mask)
 // weight chunk and multicasts it into both CTAs' rings, and each MMA warp releases a ring
 // slot in both CTAs -- the weight stream from L2 is halved, which lets Q = 2 rows per TMEM
 // buffer with NBUF = 2 buffers (epilogue overlapped with the next tile's MMAs).
-template <int M, int Q, int NBUF, int CL, bool GRID>
-__global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__ CUtensorMap tmap, const TcArgs a)
+// PAIR (one channel group): pass 1 reads the (hi, lo) receptor box -> Rhi*Whi + Rlo*Whi over 2 voxels
+// per MMA; pass 2 reads a second box whose 16-B slot x holds (Rhi(x), Rhi(x+1)), so one K = 16 MMA
+// covers 4 voxels of Rhi*Wlo (chunk LBO = 32 B): 3 MMAs per 4 voxels instead of 4.
+template <int M, int Q, int NBUF, int CL, bool PAIR, bool GRID>
+__global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__ CUtensorMap tmap,
+                                                          const __grid_constant__ CUtensorMap tmap_pair, const TcArgs a)
 {
     constexpr int KS = KSTEPS;                 // K-steps per weight-ring stage (one wait/commit per KS steps)
     constexpr unsigned STAGE = KS * WCHUNK;
@@ -236,10 +241,56 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
     if (n_tiles > 0) {
         if (warp == 0) {
             // ------------------------------------------------ TMA producer (warp-converged, one elected lane)
-            if (elect_one()) dk::prefetch_tmap(&tmap);
+            if (elect_one()) {
+                dk::prefetch_tmap(&tmap);
+                if constexpr (PAIR) dk::prefetch_tmap(&tmap_pair);
+            }
             const unsigned char* wsrc = a.W + static_cast<size_t>(block) * a.nsteps * WCHUNK;
             int ws = 0, wph = 0;                  // weight ring slot / phase
             int wuse = 0;
+            auto stream_weights = [&](int s0, int s1) {
+                for (int s = s0; s < s1; s += KS) {
+                    if (wuse >= a.wstages) dk::mbar_wait(&w_empty[ws], wph ^ 1);
+                    if (elect_one()) {
+                        dk::mbar_arrive_expect_tx(&w_full[ws], STAGE);
+                        if constexpr (CL == 1) {
+                            dk::bulk_load(w_smem + static_cast<size_t>(ws) * STAGE,
+                                          wsrc + static_cast<size_t>(s) * WCHUNK, STAGE, &w_full[ws]);
+                        } else {
+                            constexpr unsigned HALF = STAGE / CL;
+                            bulk_load_mc(w_smem + static_cast<size_t>(ws) * STAGE + crank * HALF,
+                                         wsrc + static_cast<size_t>(s) * WCHUNK + crank * HALF, HALF, &w_full[ws],
+                                         CMASK);
+                        }
+                    }
+                    __syncwarp();
+                    wuse++;
+                    if (++ws == a.wstages) {
+                        ws = 0;
+                        wph ^= 1;
+                    }
+                }
+            };
+            if constexpr (PAIR) {
+                for (int ti = 0; ti < n_tiles; ti++) {
+                    const int tile = tile_begin + ti;
+                    const int tx = tile % a.ntx, ty = (tile / a.ntx) % a.nty, tz = tile / (a.ntx * a.nty);
+                    if (ti > 0) dk::mbar_wait(&rec_empty[0], (ti - 1) & 1);
+                    if (elect_one()) {
+                        dk::mbar_arrive_expect_tx(&rec_full[0], a.box_bytes);
+                        tma_load_5d(rec_smem, &tmap, 0, tx * NT, ty * Q, tz, 0, &rec_full[0]);
+                    }
+                    __syncwarp();
+                    stream_weights(0, a.S1p);
+                    if (ti > 0) dk::mbar_wait(&rec_empty[1], (ti - 1) & 1);
+                    if (elect_one()) {
+                        dk::mbar_arrive_expect_tx(&rec_full[1], a.box_bytes);
+                        tma_load_5d(rec_smem + a.rec_stage_bytes, &tmap_pair, 0, tx * NT, ty * Q, tz, 0, &rec_full[1]);
+                    }
+                    __syncwarp();
+                    stream_weights(a.S1p, a.nsteps);
+                }
+            } else {
             for (int ti = 0; ti < n_tiles; ti++) {
                 const int tile = tile_begin + ti;
                 const int rs = ti % a.n_rec_stages, ruse = ti / a.n_rec_stages;
@@ -275,6 +326,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                     }
                 }
             }
+            }   // !PAIR
             if constexpr (CL > 1) {
                 // drain: every ring slot's last release (from both MMA warps) has arrived before exit
                 for (int i = 0; i < min(wuse, a.wstages); i++) {
@@ -293,6 +345,74 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
             const uint64_t dB0 = umma_desc(rec0, 16, 128);       // + (voxel offset >> 4)
             const uint32_t row16 = static_cast<uint32_t>(a.TXB) * 16u;
             int ws = 0, wph = 0, kin = 0;
+            // one K-step: wait for its ring stage, Q MMAs into the Q row accumulators, release the stage
+            auto issue_step = [&](uint64_t db, uint32_t dcol, uint32_t acc) {
+                if (kin == 0) {
+                    dk::mbar_wait(&w_full[ws], wph);
+                    tc_fence_after();
+                }
+                if (elect_one()) {
+                    const uint64_t da = dA0 + ((static_cast<uint32_t>(ws) * STAGE + kin * WCHUNK) >> 4);
+#pragma unroll
+                    for (int q = 0; q < Q; q++) umma_bf16(dcol + q * NT, da, db + ((q * row16) >> 4), idesc, acc);
+                    if (kin == KS - 1) {
+                        if constexpr (CL == 1) umma_commit(&w_empty[ws]);
+                        else umma_commit_mc(&w_empty[ws], CMASK);
+                    }
+                }
+                __syncwarp();
+                if (++kin == KS) {
+                    kin = 0;
+                    if (++ws == a.wstages) {
+                        ws = 0;
+                        wph ^= 1;
+                    }
+                }
+            };
+            if constexpr (PAIR) {
+                constexpr int MXQ = (M + 3) / 4;   // 4-voxel groups along x in pass 2
+                const uint64_t dP0 = umma_desc(rec0 + a.rec_stage_bytes, 32, 128);
+                for (int ti = 0; ti < n_tiles; ti++) {
+                    const int buf = ti % NBUF, buse = ti / NBUF;
+                    dk::mbar_wait(&rec_full[0], ti & 1);
+                    if (buse > 0) dk::mbar_wait(&tm_empty[buf], (buse - 1) & 1);
+                    tc_fence_after();
+                    const uint32_t dcol = tmem + static_cast<uint32_t>(buf * Q * NT);
+                    int vx = 0, vy = 0, vz = 0;
+                    for (int s = 0; s < a.S1p; s++) {   // pass 1: (Rhi, Rlo) x (Whi, Whi), voxels 2vxp, 2vxp+1
+                        const uint32_t bofs = s < a.S1 ? ((vz * a.TYB + vy) * a.TXB + 2 * vx) * 16u : 0u;
+                        issue_step(dB0 + (bofs >> 4), dcol, s > 0 ? 1u : 0u);
+                        if (++vx == MXP) {
+                            vx = 0;
+                            if (++vy == M) {
+                                vy = 0;
+                                ++vz;
+                            }
+                        }
+                    }
+                    if (elect_one()) umma_commit(&rec_empty[0]);
+                    __syncwarp();
+                    dk::mbar_wait(&rec_full[1], ti & 1);
+                    tc_fence_after();
+                    vx = vy = vz = 0;
+                    for (int s = 0; s < a.S2p; s++) {   // pass 2: (Rhi(x), Rhi(x+1)) x (Wlo, Wlo), voxels 4vxq..4vxq+3
+                        const uint32_t bofs = s < a.S2 ? ((vz * a.TYB + vy) * a.TXB + 4 * vx) * 16u : 0u;
+                        issue_step(dP0 + (bofs >> 4), dcol, 1u);
+                        if (++vx == MXQ) {
+                            vx = 0;
+                            if (++vy == M) {
+                                vy = 0;
+                                ++vz;
+                            }
+                        }
+                    }
+                    if (elect_one()) {
+                        umma_commit(&rec_empty[1]);
+                        umma_commit(&tm_full[buf]);
+                    }
+                    __syncwarp();
+                }
+            } else
             for (int ti = 0; ti < n_tiles; ti++) {
                 const int rs = ti % a.n_rec_stages, ruse = ti / a.n_rec_stages;
                 const int buf = ti % NBUF, buse = ti / NBUF;
@@ -522,6 +642,89 @@ __global__ void k_pack_weights_tc(const float* __restrict__ Lw, unsigned char* _
                     out[4 + cc] = __bfloat16_as_ushort(hi);
                 } else {
                     out[cc] = __bfloat16_as_ushort(lo);
+                }
+            }
+        }
+        uint4 pk;
+        pk.x = out[0] | (static_cast<uint32_t>(out[1]) << 16);
+        pk.y = out[2] | (static_cast<uint32_t>(out[3]) << 16);
+        pk.z = out[4] | (static_cast<uint32_t>(out[5]) << 16);
+        pk.w = out[6] | (static_cast<uint32_t>(out[7]) << 16);
+        reinterpret_cast<uint4*>(W)[i] = pk;
+    }
+}
+
+// PAIR scheme, second receptor copy: slot X holds (Rhi_0..3(X), Rhi_0..3(X+1)) of channels 0..3.
+__global__ void k_pack_receptor_pair_tc(const float* __restrict__ R, uint16_t* __restrict__ Rb, int nx, int ny, int nz,
+                                        int Xp, int Yp, int Zp, int P)
+{
+    const size_t total = static_cast<size_t>(Zp) * Yp * Xp;
+    for (size_t i = blockIdx.x * static_cast<size_t>(blockDim.x) + threadIdx.x; i < total;
+         i += static_cast<size_t>(gridDim.x) * blockDim.x) {
+        const int X = static_cast<int>(i % Xp);
+        size_t rr = i / Xp;
+        const int Y = static_cast<int>(rr % Yp);
+        const int Z = static_cast<int>(rr / Yp);
+        uint16_t out[8];
+#pragma unroll
+        for (int c = 0; c < 8; c++) {
+            const int p = c & 3, dx = c >> 2;
+            float f = 0.f;
+            if (p < P) f = R[((static_cast<size_t>(p) * nz + Z % nz) * ny + Y % ny) * nx + (X + dx) % nx];
+            out[c] = __bfloat16_as_ushort(__float2bfloat16_rn(f));
+        }
+        uint4 pk;
+        pk.x = out[0] | (static_cast<uint32_t>(out[1]) << 16);
+        pk.y = out[2] | (static_cast<uint32_t>(out[3]) << 16);
+        pk.z = out[4] | (static_cast<uint32_t>(out[5]) << 16);
+        pk.w = out[6] | (static_cast<uint32_t>(out[7]) << 16);
+        reinterpret_cast<uint4*>(Rb)[i] = pk;
+    }
+}
+
+// PAIR scheme A operand: steps [0, S1p) = pass 1 chunks (Whi(vx), Whi(vx)), vx = 2 vxp + c;
+// steps [S1p, S1p + S2p) = pass 2 chunks (Wlo(vx0), Wlo(vx0 + 1)), vx0 = 4 vxq + 2c; padding = 0.
+__global__ void k_pack_weights_tc_pair(const float* __restrict__ Lw, unsigned char* __restrict__ W, int n_slots, int P,
+                                       int m, int S1, int S1p, int S2, int S2p)
+{
+    const int MXP = (m + 1) / 2, MXQ = (m + 3) / 4, m3 = m * m * m, nsteps = S1p + S2p;
+    const long long n_blocks = (n_slots + ROT - 1) / ROT;
+    const long long total = n_blocks * nsteps * 2 * ROT;
+    for (long long i = blockIdx.x * static_cast<long long>(blockDim.x) + threadIdx.x; i < total;
+         i += static_cast<long long>(gridDim.x) * blockDim.x) {
+        const int r = static_cast<int>(i % ROT);
+        const int c = static_cast<int>((i / ROT) % 2);
+        const int s = static_cast<int>((i / (2 * ROT)) % nsteps);
+        const long long blk = i / (2LL * ROT * nsteps);
+        const long long slot = blk * ROT + r;
+        uint16_t out[8] = {0, 0, 0, 0, 0, 0, 0, 0};
+        auto wval = [&](int vz, int vy, int vx, int p) -> float {
+            if (vx >= m || p >= P) return 0.f;
+            const int v = (vz * m + vy) * m + vx;
+            return Lw[((static_cast<size_t>(slot / dk::RB) * P + p) * m3 + v) * dk::RB + slot % dk::RB];
+        };
+        if (slot < n_slots) {
+            if (s < S1) {
+                const int vxp = s % MXP, vy = (s / MXP) % m, vz = s / (MXP * m);
+                const int vx = 2 * vxp + c;
+#pragma unroll
+                for (int p = 0; p < 4; p++) {
+                    const __nv_bfloat16 hi = __float2bfloat16_rn(wval(vz, vy, vx, p));
+                    out[p] = out[4 + p] = __bfloat16_as_ushort(hi);
+                }
+            } else if (s >= S1p && s - S1p < S2) {
+                const int t = s - S1p;
+                const int vxq = t % MXQ, vy = (t / MXQ) % m, vz = t / (MXQ * m);
+                const int vx0 = 4 * vxq + 2 * c;
+#pragma unroll
+                for (int p = 0; p < 4; p++) {
+#pragma unroll
+                    for (int d = 0; d < 2; d++) {
+                        const float f = wval(vz, vy, vx0 + d, p);
+                        const __nv_bfloat16 hi = __float2bfloat16_rn(f);
+                        const __nv_bfloat16 lo = __float2bfloat16_rn(f - __bfloat162float(hi));
+                        out[4 * d + p] = __bfloat16_as_ushort(lo);
+                    }
                 }
             }
         }
