@@ -190,13 +190,14 @@ def roofline(pk, pk_kind, info, c, flops_launch, corr_ms, ms_step, units_local):
     148 SMs x 128 lanes x 2 x clock; tcgen05 engine -> bound "tensor" against the measured bf16
     dense peak (the kernel's own operand dtype).  ``achieved`` always uses the ALGORITHMIC
     dense correlation FLOPs 2*P*m^3*N^3 per unit; the tcgen05 engine executes 4x that (bf16x3
-    split: 2 passes x 8 bf16 lanes per 4 channels) plus x-pair padding for odd m."""
+    split) -- 3x with the PAIR scheme, 4x without -- plus x-padding for odd m (from dock_get_info)."""
     n_sms = int(info["n_sms"])
     achieved = flops_launch / (corr_ms / 1000.0) / 1e12
     if info["engine_last"] == 2:
         peak = float(pk.get("bf16_tflops", 1590.0))
-        mx = (c.m + 1) // 2 * 2
-        executed = flops_launch * 4.0 * mx / c.m
+        ks = int(info.get("tc_ksteps_last", 0)) or 2 * c.m * c.m * ((c.m + 1) // 2)
+        # executed bf16 MMA FLOPs: K = 16 per step, ks steps per translation row (bf16x3 split + padding)
+        executed = flops_launch * (ks * 16.0) / (c.P * c.m ** 3)
         v = int(info.get("tc_variant_last", 1)) or 1
         kname = f"k_corr_tc<{c.m},4,1,1,false>" if v == 1 else f"k_corr_tc<{c.m},2,2,2,false>"
         return {"bound": "tensor", "engine": f"tcgen05 bf16x3 (variant {v})", "kernel": kname,

@@ -158,6 +158,7 @@ typedef struct {
     int engine_last;           /* engine of the last correlation: 1 FP32 FFMA, 2 tcgen05 bf16x3 */
     int tc_available;          /* 1 if the tcgen05 engine is available for m_max */
     int tc_variant_last;       /* tcgen05 variant of the last correlation (1 or 2), 0 if FFMA */
+    int tc_ksteps_last;        /* K-steps (K = 16 each) per translation row executed by the last tcgen05 launch */
 } dock_info;
 
 dock_status dock_get_info(const dock_ctx* ctx, dock_info* info);

@@ -69,6 +69,7 @@ struct dock_ctx {
     int engine_last = 0;
     int tc_variant = 0;        // DOCK_TUNE_TC_VARIANT: 0 auto, 1 (Q4, 1 TMEM buffer), 2 (Q2, 2 buffers, CTA pair)
     int tc_variant_last = 0;
+    int tc_ksteps_last = 0;   // K-steps (of 16) per translation row in the last tcgen05 launch
     uint16_t* d_rec_tc = nullptr;
     uint16_t* d_rec_pair = nullptr;   // PAIR-scheme receptor copy (P <= 4)
     int tc_Gch = 0, tc_ntx = 0, tc_ntz = 0, tc_Xp = 0, tc_Yp = 0, tc_Zp = 0;
@@ -283,9 +284,14 @@ dock_status make_tc_plan(dock_ctx* ctx, int m, int v)
 {
     TcPlan& pl = ctx->tcplan[v][m];
     if (pl.ok || !ctx->d_rec_tc) return DOCK_OK;
-    pl.pair = ctx->tc_Gch == 1 && ctx->d_rec_pair != nullptr;
-    if (!pl.pair && v != 1) return DOCK_OK;          // the CTA-pair variant is built for the PAIR scheme only
     const int KS = tc::KSTEPS;
+    const int budget = kSmemLimit - 2048;   // static shared memory (barriers) and slack
+    const int stage = KS * tc::WCHUNK;
+    const int min_ring = 3 * stage;
+    // PAIR needs the (hi,lo) box and the (hi,hi') box resident together; otherwise the 2-pass scheme
+    const int pair_box = round_up(16 * tc_txb_any(m) * (tc_q(v) + m - 1) * m, 1024);
+    pl.pair = ctx->tc_Gch == 1 && ctx->d_rec_pair != nullptr && 2 * pair_box + min_ring <= budget;
+    if (!pl.pair && v != 1) return DOCK_OK;          // the CTA-pair variant is built for the PAIR scheme only
     pl.TXB = pl.pair ? tc_txb_any(m) : tc_txb(m);
     pl.TYB = tc_q(v) + m - 1;
     pl.TZB = m;
@@ -300,9 +306,6 @@ dock_status make_tc_plan(dock_ctx* ctx, int m, int v)
     } else {
         pl.nsteps = ctx->tc_Gch * 2 * m * m * ((m + 1) / 2);
     }
-    const int budget = kSmemLimit - 2048;   // static shared memory (barriers) and slack
-    const int stage = KS * tc::WCHUNK;
-    const int min_ring = 3 * stage;
     if (2 * pl.rec_stage_bytes + min_ring <= budget) pl.n_rec_stages = 2;
     else if (!pl.pair && pl.rec_stage_bytes + min_ring <= budget) pl.n_rec_stages = 1;
     else return DOCK_OK;                    // this m is not eligible for the tensor-core engine
@@ -1005,6 +1008,7 @@ dock_status dock_get_info(const dock_ctx* ctx, dock_info* info)
     info->engine_last = ctx->engine_last;
     info->tc_available = (ctx->tcplan[1][ctx->m_max].ok || ctx->tcplan[2][ctx->m_max].ok) ? 1 : 0;
     info->tc_variant_last = ctx->tc_variant_last;
+    info->tc_ksteps_last = ctx->tc_ksteps_last;
     return DOCK_OK;
 }
 
@@ -1084,6 +1088,7 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
         if (!plan_tc_launch(ctx, m, n_units, &v, &G)) return fail(ctx, DOCK_E_UNSUPPORTED, "no tensor-core plan");
         TRY(pack_weights_tc(ctx, m, ctx->tcplan[v][m], n_units, static_cast<const float*>(ctx->Lw.p)));
         ctx->tc_variant_last = v;
+        ctx->tc_ksteps_last = ctx->tcplan[v][m].nsteps;
         tc::TcArgs ta = tc_args(ctx, m, v, n_units, G, static_cast<const unsigned char*>(ctx->Wtc.p));
         ta.k = k;
         ta.rho = rho;
