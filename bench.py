@@ -51,6 +51,7 @@ def parse():
     ap.add_argument("--engine", default="auto", choices=["auto", "ffma", "tc"],
                     help="correlation engine: auto (tcgen05 when eligible), ffma (FP32 FFMA), tc (tcgen05 bf16x3)")
     ap.add_argument("--no-alt", action="store_true", help="skip the secondary measurement of the other engine")
+    ap.add_argument("--tc-epi", type=int, default=0, choices=[0, 4, 8, 16], help="tcgen05 epilogue warps (0 auto)")
     ap.add_argument("--tc-variant", type=int, default=0, choices=[0, 1, 2],
                     help="tcgen05 tiling: 0 auto, 1 = 4 rows x 1 TMEM buffer, 2 = CTA pair, 2 rows x 2 buffers")
     return ap.parse_args()
@@ -243,6 +244,7 @@ def run_ours(args):
     ENG = {"auto": 0, "ffma": 1, "tc": 2}
     D.dock_set_tuning(ctx, D.DOCK_TUNE_ENGINE, ENG[args.engine])
     D.dock_set_tuning(ctx, D.DOCK_TUNE_TC_VARIANT, args.tc_variant)
+    D.dock_set_tuning(ctx, 6, args.tc_epi)   # DOCK_TUNE_TC_EPILOGUE_WARPS
     probes_dev = [{"xyz": torch.from_numpy(p.xyz).to(dev), "coef": torch.from_numpy(p.coef).to(dev), "m": p.m}
                   for p in probes]
     rot_dev = torch.from_numpy(rot).to(dev)

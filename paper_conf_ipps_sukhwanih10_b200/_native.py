@@ -23,6 +23,7 @@ DOCK_TUNE_FORCE_FALLBACK = 2
 DOCK_TUNE_CAND_CAP = 3
 DOCK_TUNE_ENGINE = 4
 DOCK_TUNE_TC_VARIANT = 5
+DOCK_TUNE_TC_EPILOGUE_WARPS = 6
 
 STATUS_NAMES = {0: "DOCK_OK", -1: "DOCK_E_INVALID_ARG", -2: "DOCK_E_UNSUPPORTED",
                 -3: "DOCK_E_PROBE_OUTSIDE_GRID", -4: "DOCK_E_BAD_ROTATION", -5: "DOCK_E_CUDA",

@@ -69,7 +69,8 @@ struct dock_ctx {
     int engine_last = 0;
     int tc_variant = 0;        // DOCK_TUNE_TC_VARIANT: 0 auto, 1 (Q4, 1 TMEM buffer), 2 (Q2, 2 buffers, CTA pair)
     int tc_variant_last = 0;
-    int tc_ksteps_last = 0;   // K-steps (of 16) per translation row in the last tcgen05 launch
+    int tc_ksteps_last = 0;
+    int tc_nepi = 0;          // epilogue warps (0 = one row per thread)   // K-steps (of 16) per translation row in the last tcgen05 launch
     uint16_t* d_rec_tc = nullptr;
     uint16_t* d_rec_pair = nullptr;   // PAIR-scheme receptor copy (P <= 4)
     int tc_Gch = 0, tc_ntx = 0, tc_ntz = 0, tc_Xp = 0, tc_Yp = 0, tc_Zp = 0;
@@ -305,6 +306,7 @@ dock_status make_tc_plan(dock_ctx* ctx, int m, int v)
         pl.nsteps = pl.S1p + pl.S2p;
     } else {
         pl.nsteps = ctx->tc_Gch * 2 * m * m * ((m + 1) / 2);
+        if (pl.nsteps % KS) return DOCK_OK;   // the 2-pass scheme needs whole ring stages
     }
     if (2 * pl.rec_stage_bytes + min_ring <= budget) pl.n_rec_stages = 2;
     else if (!pl.pair && pl.rec_stage_bytes + min_ring <= budget) pl.n_rec_stages = 1;
@@ -339,11 +341,11 @@ cudaError_t launch_tc_t(const TcPlan& pl, const tc::TcArgs& a, int grid, cudaStr
     cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, pl.smem);
     if (e != cudaSuccess) return e;
     if constexpr (CL == 1) {
-        kern<<<grid, tc::NTHREADS, pl.smem, st>>>(pl.tmap, pl.tmap_pair, a);
+        kern<<<grid, (2 + a.nepi) * 32, pl.smem, st>>>(pl.tmap, pl.tmap_pair, a);
     } else {
         cudaLaunchConfig_t cfg{};
         cfg.gridDim = dim3(grid);
-        cfg.blockDim = dim3(tc::NTHREADS);
+        cfg.blockDim = dim3((2 + a.nepi) * 32);
         cfg.dynamicSmemBytes = pl.smem;
         cfg.stream = st;
         cudaLaunchAttribute at[1];
@@ -687,6 +689,7 @@ tc::TcArgs tc_args(dock_ctx* ctx, int m, int v, int n_slots, int G, const unsign
     a.rec_stage_bytes = tp.rec_stage_bytes;
     a.n_rec_stages = tp.n_rec_stages;
     a.wstages = tp.wstages;
+    a.nepi = ctx->tc_nepi > 0 ? std::min(4 * tc_q(v), ctx->tc_nepi) : 4 * tc_q(v);   // one row per thread
     a.S1 = tp.S1;
     a.S1p = tp.S1p;
     a.S2 = tp.S2;
@@ -966,6 +969,11 @@ dock_status dock_set_tuning(dock_ctx* ctx, int key, int64_t value)
         case DOCK_TUNE_TC_VARIANT:
             if (value < 0 || value > 2) return fail(ctx, DOCK_E_INVALID_ARG, "tc variant must be 0, 1 or 2");
             ctx->tc_variant = (int)value;
+            return DOCK_OK;
+        case DOCK_TUNE_TC_EPILOGUE_WARPS:
+            if (value != 0 && value != 4 && value != 8 && value != 16)
+                return fail(ctx, DOCK_E_INVALID_ARG, "epilogue warps must be 0, 4, 8 or 16");
+            ctx->tc_nepi = (int)value;
             return DOCK_OK;
         case DOCK_TUNE_CAND_CAP:
             if (value < 32 || value > (1 << 20)) return fail(ctx, DOCK_E_INVALID_ARG, "cand cap out of range");

@@ -29,12 +29,12 @@ using dk::KEY_MAX;
 
 constexpr int ROT = 128;        // rotations per block (MMA M)
 constexpr int NT = 128;         // translations per row (MMA N)
-constexpr int NEPI = 8;         // epilogue warps (2 per TMEM lane quarter)
-constexpr int NTHREADS = (2 + NEPI) * 32;
+constexpr int NEPI_MAX = 16;    // epilogue warps: a.nepi in {4, 8, 16} (1, 2 or 4 per TMEM lane quarter)
+constexpr int NTHREADS = (2 + NEPI_MAX) * 32;   // launch bound; the launch uses (2 + a.nepi) * 32 threads
 constexpr int WSTAGES = 16;     // max weight ring depth (runtime a.wstages <= 16; 16 x 4 KB covers the L2 latency)
 constexpr int WCHUNK = 2 * ROT * 16;   // bytes of one K-step of A (2 K-chunks x 128 rotations x 16 B)
-constexpr int KSTEPS = 2;       // K-steps of A per ring stage (nsteps is always even: 2 passes)
-constexpr int LIST = 32;        // per-thread candidate list (exact top-LIST keys of one rotation)
+constexpr int KSTEPS = 4;       // K-steps of A per ring stage (one elected issue block of KSTEPS*Q MMAs)
+constexpr int LIST = 16;        // per-thread candidate list (exact top-LIST keys of one rotation and row class)
 
 struct TcArgs {
     int nx, ny, nz;
@@ -48,7 +48,8 @@ struct TcArgs {
     int box_bytes;              // one channel group's receptor box
     int rec_stage_bytes;        // G_ch * box_bytes rounded to 1024
     int n_rec_stages;           // 1 or 2
-    int wstages;                // weight ring depth (4..WSTAGES)
+    int wstages;                // weight ring depth (3..WSTAGES)
+    int nepi;                   // epilogue warps (4, 8 or 16)
     // top-k
     int k, rho, cap;
     unsigned long long* T;
@@ -220,7 +221,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
         }
         for (int i = 0; i < NBUF; i++) {
             dk::mbar_init(&tm_full[i], 1);
-            dk::mbar_init(&tm_empty[i], NEPI);
+            dk::mbar_init(&tm_empty[i], a.nepi);
         }
         dk::fence_mbar_init();
     }
@@ -339,136 +340,92 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
             }
         } else if (warp == 1) {
             // ------------------------------------------------ MMA issuer (warp-converged, one elected lane)
+            // One elected block per ring stage (KS K-steps x Q rows = KS*Q MMAs): the warp re-converges
+            // once per stage, not once per K-step (the re-convergence waits for the tcgen05 issue).
             constexpr uint32_t idesc = umma_idesc(ROT, NT);
+            constexpr int MXQ = (M + 3) / 4;   // PAIR pass 2: 4-voxel groups along x
             const uint32_t rec0 = dk::smem_u32(rec_smem), w0 = dk::smem_u32(w_smem);
-            const uint64_t dA0 = umma_desc(w0, ROT * 16, 128);   // + (slot offset >> 4)
-            const uint64_t dB0 = umma_desc(rec0, 16, 128);       // + (voxel offset >> 4)
+            const uint64_t dA0 = umma_desc(w0, ROT * 16, 128);                      // + (slot offset >> 4)
+            const uint64_t dB0 = umma_desc(rec0, 16, 128);                          // + (voxel offset >> 4)
+            const uint64_t dP0 = umma_desc(rec0 + (PAIR ? a.rec_stage_bytes : 0), 32, 128);
             const uint32_t row16 = static_cast<uint32_t>(a.TXB) * 16u;
-            int ws = 0, wph = 0, kin = 0;
-            // one K-step: wait for its ring stage, Q MMAs into the Q row accumulators, release the stage
-            auto issue_step = [&](uint64_t db, uint32_t dcol, uint32_t acc) {
-                if (kin == 0) {
-                    dk::mbar_wait(&w_full[ws], wph);
-                    tc_fence_after();
+            const uint32_t rowTY = static_cast<uint32_t>(a.TYB) * row16;
+            int ws = 0, wph = 0;
+            // B descriptor of K-step s: PAIR pass 1 (kind 0), PAIR pass 2 (kind 1) or the 2-pass scheme (kind 2)
+            auto bdesc = [&](int kind, int s, uint32_t rofs) -> uint64_t {
+                if (kind == 0) {
+                    if (s >= a.S1) return dB0;
+                    const int vxp = s % MXP, vy = (s / MXP) % M, vz = s / (MXP * M);
+                    return dB0 + ((rofs + vz * rowTY + vy * row16 + vxp * 32u) >> 4);
                 }
+                if (kind == 1) {
+                    if (s >= a.S2) return dP0;
+                    const int vxq = s % MXQ, vy = (s / MXQ) % M, vz = s / (MXQ * M);
+                    return dP0 + ((vz * rowTY + vy * row16 + vxq * 64u) >> 4);
+                }
+                const int vxp = s % MXP, vy = (s / MXP) % M, vz = (s / (MXP * M)) % M;
+                const int g = s / (MXP * M * M * 2);
+                return dB0 + ((rofs + g * a.box_bytes + vz * rowTY + vy * row16 + vxp * 32u) >> 4);
+            };
+            auto issue_stage = [&](int kind, int s0, uint32_t rofs, uint32_t dcol, bool first) {
+                dk::mbar_wait(&w_full[ws], wph);
+                tc_fence_after();
                 if (elect_one()) {
-                    const uint64_t da = dA0 + ((static_cast<uint32_t>(ws) * STAGE + kin * WCHUNK) >> 4);
+                    const uint64_t da0 = dA0 + ((static_cast<uint32_t>(ws) * STAGE) >> 4);
 #pragma unroll
-                    for (int q = 0; q < Q; q++) umma_bf16(dcol + q * NT, da, db + ((q * row16) >> 4), idesc, acc);
-                    if (kin == KS - 1) {
-                        if constexpr (CL == 1) umma_commit(&w_empty[ws]);
-                        else umma_commit_mc(&w_empty[ws], CMASK);
+                    for (int ks = 0; ks < KS; ks++) {
+                        const uint64_t db = bdesc(kind, s0 + ks, rofs);
+                        const uint64_t da = da0 + ((ks * WCHUNK) >> 4);
+#pragma unroll
+                        for (int q = 0; q < Q; q++)
+                            umma_bf16(dcol + q * NT, da, db + ((q * row16) >> 4), idesc, (first && ks == 0) ? 0u : 1u);
                     }
+                    if constexpr (CL == 1) umma_commit(&w_empty[ws]);
+                    else umma_commit_mc(&w_empty[ws], CMASK);
                 }
                 __syncwarp();
-                if (++kin == KS) {
-                    kin = 0;
-                    if (++ws == a.wstages) {
-                        ws = 0;
-                        wph ^= 1;
-                    }
+                if (++ws == a.wstages) {
+                    ws = 0;
+                    wph ^= 1;
                 }
             };
-            if constexpr (PAIR) {
-                constexpr int MXQ = (M + 3) / 4;   // 4-voxel groups along x in pass 2
-                const uint64_t dP0 = umma_desc(rec0 + a.rec_stage_bytes, 32, 128);
-                for (int ti = 0; ti < n_tiles; ti++) {
-                    const int buf = ti % NBUF, buse = ti / NBUF;
+            for (int ti = 0; ti < n_tiles; ti++) {
+                const int buf = ti % NBUF, buse = ti / NBUF;
+                const uint32_t dcol = tmem + static_cast<uint32_t>(buf * Q * NT);
+                if constexpr (PAIR) {
                     dk::mbar_wait(&rec_full[0], ti & 1);
                     if (buse > 0) dk::mbar_wait(&tm_empty[buf], (buse - 1) & 1);
                     tc_fence_after();
-                    const uint32_t dcol = tmem + static_cast<uint32_t>(buf * Q * NT);
-                    int vx = 0, vy = 0, vz = 0;
-                    for (int s = 0; s < a.S1p; s++) {   // pass 1: (Rhi, Rlo) x (Whi, Whi), voxels 2vxp, 2vxp+1
-                        const uint32_t bofs = s < a.S1 ? ((vz * a.TYB + vy) * a.TXB + 2 * vx) * 16u : 0u;
-                        issue_step(dB0 + (bofs >> 4), dcol, s > 0 ? 1u : 0u);
-                        if (++vx == MXP) {
-                            vx = 0;
-                            if (++vy == M) {
-                                vy = 0;
-                                ++vz;
-                            }
-                        }
-                    }
+                    for (int s = 0; s < a.S1p; s += KS) issue_stage(0, s, 0u, dcol, s == 0);
                     if (elect_one()) umma_commit(&rec_empty[0]);
                     __syncwarp();
                     dk::mbar_wait(&rec_full[1], ti & 1);
                     tc_fence_after();
-                    vx = vy = vz = 0;
-                    for (int s = 0; s < a.S2p; s++) {   // pass 2: (Rhi(x), Rhi(x+1)) x (Wlo, Wlo), voxels 4vxq..4vxq+3
-                        const uint32_t bofs = s < a.S2 ? ((vz * a.TYB + vy) * a.TXB + 4 * vx) * 16u : 0u;
-                        issue_step(dP0 + (bofs >> 4), dcol, 1u);
-                        if (++vx == MXQ) {
-                            vx = 0;
-                            if (++vy == M) {
-                                vy = 0;
-                                ++vz;
-                            }
-                        }
-                    }
+                    for (int s = 0; s < a.S2p; s += KS) issue_stage(1, s, 0u, dcol, false);
                     if (elect_one()) {
                         umma_commit(&rec_empty[1]);
                         umma_commit(&tm_full[buf]);
                     }
                     __syncwarp();
-                }
-            } else
-            for (int ti = 0; ti < n_tiles; ti++) {
-                const int rs = ti % a.n_rec_stages, ruse = ti / a.n_rec_stages;
-                const int buf = ti % NBUF, buse = ti / NBUF;
-                dk::mbar_wait(&rec_full[rs], ruse & 1);
-                if (buse > 0) dk::mbar_wait(&tm_empty[buf], (buse - 1) & 1);
-                tc_fence_after();
-                const uint32_t dcol = tmem + static_cast<uint32_t>(buf * Q * NT);
-                uint32_t acc = 0;
-                for (int g = 0; g < a.G_ch; g++) {
-                    const uint32_t gofs = static_cast<uint32_t>(rs * a.rec_stage_bytes + g * a.box_bytes);
-                    for (int pass = 0; pass < 2; pass++) {
-                        for (int vz = 0; vz < M; vz++) {
-                            for (int vy = 0; vy < M; vy++) {
-                                const uint32_t rowofs = gofs + static_cast<uint32_t>(vz * a.TYB + vy) * row16;
-#pragma unroll
-                                for (int vxp = 0; vxp < MXP; vxp++) {
-                                    if (kin == 0) {
-                                        dk::mbar_wait(&w_full[ws], wph);
-                                        tc_fence_after();
-                                    }
-                                    if (elect_one()) {
-                                        const uint64_t da =
-                                            dA0 + ((static_cast<uint32_t>(ws) * STAGE + kin * WCHUNK) >> 4);
-                                        const uint64_t db = dB0 + ((rowofs + vxp * 32u) >> 4);
-#pragma unroll
-                                        for (int q = 0; q < Q; q++)
-                                            umma_bf16(dcol + q * NT, da, db + ((q * row16) >> 4), idesc, acc);
-                                        if (kin == KS - 1) {
-                                            if constexpr (CL == 1) umma_commit(&w_empty[ws]);
-                                            else umma_commit_mc(&w_empty[ws], CMASK);
-                                        }
-                                    }
-                                    __syncwarp();
-                                    acc = 1;
-                                    if (++kin == KS) {
-                                        kin = 0;
-                                        if (++ws == a.wstages) {
-                                            ws = 0;
-                                            wph ^= 1;
-                                        }
-                                    }
-                                }
-                            }
-                        }
+                } else {
+                    const int rs = ti % a.n_rec_stages, ruse = ti / a.n_rec_stages;
+                    dk::mbar_wait(&rec_full[rs], ruse & 1);
+                    if (buse > 0) dk::mbar_wait(&tm_empty[buf], (buse - 1) & 1);
+                    tc_fence_after();
+                    const uint32_t rofs = static_cast<uint32_t>(rs * a.rec_stage_bytes);
+                    for (int s = 0; s < a.nsteps; s += KS) issue_stage(2, s, rofs, dcol, s == 0);
+                    if (elect_one()) {
+                        umma_commit(&tm_full[buf]);
+                        umma_commit(&rec_empty[rs]);
                     }
+                    __syncwarp();
                 }
-                if (elect_one()) {
-                    umma_commit(&tm_full[buf]);
-                    umma_commit(&rec_empty[rs]);
-                }
-                __syncwarp();
             }
         } else {
             // ------------------------------------------------ epilogue warps
             const int quarter = warp & 3;
-            const int half = (warp - 2) >> 2;
+            const int half = (warp - 2) >> 2;         // row class of this warp
+            const int nclass = a.nepi >> 2;
             const int r = quarter * 32 + lane;                  // rotation within the block (TMEM lane)
             const int slot = block * ROT + r;
             const bool rot_ok = slot < a.n_slots;
@@ -483,7 +440,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                 dk::mbar_wait(&tm_full[buf], buse & 1);
                 tc_fence_after();
                 const int tx = tile % a.ntx, ty = (tile / a.ntx) % a.nty, tz = tile / (a.ntx * a.nty);
-                for (int q = half; q < Q; q += 2) {
+                for (int q = half; q < Q; q += nclass) {
                     const int y = ty * Q + q, z = tz;
                     const bool row_ok = rot_ok && y < a.ny && z < a.nz;
                     const int x0 = tx * NT;
