@@ -288,7 +288,7 @@ dock_status make_tc_plan(dock_ctx* ctx, int m, int v)
     const int KS = tc::KSTEPS;
     const int budget = kSmemLimit - 2048;   // static shared memory (barriers) and slack
     const int stage = KS * tc::WCHUNK;
-    const int min_ring = 3 * stage;
+    const int min_ring = 2 * stage;
     // PAIR needs the (hi,lo) box and the (hi,hi') box resident together; otherwise the 2-pass scheme
     const int pair_box = round_up(16 * tc_txb_any(m) * (tc_q(v) + m - 1) * m, 1024);
     pl.pair = ctx->tc_Gch == 1 && ctx->d_rec_pair != nullptr && 2 * pair_box + min_ring <= budget;
