@@ -74,7 +74,7 @@ struct dock_ctx {
     uint16_t* d_rec_tc = nullptr;
     uint16_t* d_rec_pair = nullptr;   // PAIR-scheme receptor copy (P <= 4)
     int tc_Gch = 0, tc_ntx = 0, tc_ntz = 0, tc_Xp = 0, tc_Yp = 0, tc_Zp = 0;
-    TcPlan tcplan[3][DOCK_MAX_M + 1];   // [variant][m]
+    TcPlan tcplan[4][DOCK_MAX_M + 1];   // [variant][m]
     DevBuf Wtc;
     // per-call scratch (grow-only)
     DevBuf xyz, coef, off, rot, Lw, T, mu, cnt, cand, poses, fb_list, grid, slots, units, Lw_fb, picks;
@@ -274,8 +274,11 @@ cudaError_t launch_corr(int m, const MPlan& pl, const dk::CorrArgs& a, int grid,
 
 int tc_txb(int m) { return tc::NT + (m + 1) / 2 * 2 - 1; }
 // tcgen05 variants: 1 = Q4 rows x 1 TMEM buffer, single CTA; 2 = Q2 rows x 2 buffers, CTA pair + multicast.
-inline int tc_q(int v) { return v == 1 ? 4 : 2; }
+// tile rows (translation rows per tile): variants 1 and 3 tile 4 rows, variant 2 tiles 2
+inline int tc_q(int v) { return v == 2 ? 2 : 4; }
 inline int tc_cl(int v) { return v == 1 ? 1 : 2; }
+// receptor rows held per CTA (variant 3 splits the 4 tile rows over the CTA pair)
+inline int tc_rows_cta(int v) { return v == 1 ? 4 : 2; }
 inline int tc_nty(const dock_ctx* c, int v) { return (c->ny + tc_q(v) - 1) / tc_q(v); }
 inline int tc_ntiles(const dock_ctx* c, int v) { return c->tc_ntx * tc_nty(c, v) * c->tc_ntz; }
 
@@ -290,11 +293,11 @@ dock_status make_tc_plan(dock_ctx* ctx, int m, int v)
     const int stage = KS * tc::WCHUNK;
     const int min_ring = 2 * stage;
     // PAIR needs the (hi,lo) box and the (hi,hi') box resident together; otherwise the 2-pass scheme
-    const int pair_box = round_up(16 * tc_txb_any(m) * (tc_q(v) + m - 1) * m, 1024);
+    const int pair_box = round_up(16 * tc_txb_any(m) * (tc_rows_cta(v) + m - 1) * m, 1024);
     pl.pair = ctx->tc_Gch == 1 && ctx->d_rec_pair != nullptr && 2 * pair_box + min_ring <= budget;
-    if (!pl.pair && v != 1) return DOCK_OK;          // the CTA-pair variant is built for the PAIR scheme only
+    if (!pl.pair && v != 1) return DOCK_OK;          // the CTA-pair variants are built for the PAIR scheme only
     pl.TXB = pl.pair ? tc_txb_any(m) : tc_txb(m);
-    pl.TYB = tc_q(v) + m - 1;
+    pl.TYB = tc_rows_cta(v) + m - 1;
     pl.TZB = m;
     pl.box_bytes = 16 * pl.TXB * pl.TYB * pl.TZB;
     pl.rec_stage_bytes = round_up(ctx->tc_Gch * pl.box_bytes, 1024);
@@ -378,9 +381,49 @@ cudaError_t launch_tc_v(int m, const TcPlan& pl, const tc::TcArgs& a, int grid, 
     }
 }
 
+template <int M, bool GRID>
+cudaError_t launch_tc2_t(const TcPlan& pl, const tc::TcArgs& a, int grid, cudaStream_t st)
+{
+    auto kern = tc::k_corr_tc2<M, GRID>;
+    cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, pl.smem);
+    if (e != cudaSuccess) return e;
+    cudaLaunchConfig_t cfg{};
+    cfg.gridDim = dim3(grid);
+    cfg.blockDim = dim3((2 + a.nepi) * 32);
+    cfg.dynamicSmemBytes = pl.smem;
+    cfg.stream = st;
+    cudaLaunchAttribute at[1];
+    at[0].id = cudaLaunchAttributeClusterDimension;
+    at[0].val.clusterDim.x = 2;
+    at[0].val.clusterDim.y = 1;
+    at[0].val.clusterDim.z = 1;
+    cfg.attrs = at;
+    cfg.numAttrs = 1;
+    e = cudaLaunchKernelEx(&cfg, kern, pl.tmap, pl.tmap_pair, a);
+    if (e != cudaSuccess) return e;
+    return cudaGetLastError();
+}
+
+template <bool GRID>
+cudaError_t launch_tc2(int m, const TcPlan& pl, const tc::TcArgs& a, int grid, cudaStream_t st)
+{
+    switch (m) {
+        case 1: return launch_tc2_t<1, GRID>(pl, a, grid, st);
+        case 2: return launch_tc2_t<2, GRID>(pl, a, grid, st);
+        case 3: return launch_tc2_t<3, GRID>(pl, a, grid, st);
+        case 4: return launch_tc2_t<4, GRID>(pl, a, grid, st);
+        case 5: return launch_tc2_t<5, GRID>(pl, a, grid, st);
+        case 6: return launch_tc2_t<6, GRID>(pl, a, grid, st);
+        case 7: return launch_tc2_t<7, GRID>(pl, a, grid, st);
+        case 8: return launch_tc2_t<8, GRID>(pl, a, grid, st);
+        default: return cudaErrorInvalidValue;
+    }
+}
+
 template <bool GRID>
 cudaError_t launch_tc(int m, int v, const TcPlan& pl, const tc::TcArgs& a, int grid, cudaStream_t st)
 {
+    if (v == 3) return launch_tc2<GRID>(m, pl, a, grid, st);
     if (!pl.pair) return v == 1 ? launch_tc_v<1, false, GRID>(m, pl, a, grid, st) : cudaErrorInvalidValue;
     return v == 1 ? launch_tc_v<1, true, GRID>(m, pl, a, grid, st) : launch_tc_v<2, true, GRID>(m, pl, a, grid, st);
 }
@@ -689,7 +732,7 @@ tc::TcArgs tc_args(dock_ctx* ctx, int m, int v, int n_slots, int G, const unsign
     a.rec_stage_bytes = tp.rec_stage_bytes;
     a.n_rec_stages = tp.n_rec_stages;
     a.wstages = tp.wstages;
-    a.nepi = ctx->tc_nepi > 0 ? std::min(4 * tc_q(v), ctx->tc_nepi) : 4 * tc_q(v);   // one row per thread
+    a.nepi = ctx->tc_nepi > 0 ? std::min(16, ctx->tc_nepi) : (v == 2 ? 8 : 16);   // one row per thread
     a.S1 = tp.S1;
     a.S1p = tp.S1p;
     a.S2 = tp.S2;
@@ -711,6 +754,15 @@ bool plan_tc_launch(dock_ctx* ctx, int m, int n_slots, int* v_out, int* G_out)
             *G_out = G;
             return true;
         }
+    }
+    if (ctx->tc_variant == 3 && ctx->tcplan[3][m].ok) {
+        // CTA pairs over pairs of rotation blocks; a pair occupies two SMs
+        const int64_t n_pairs = (n_blocks + 1) / 2;
+        dock_ctx tmp = *ctx;
+        tmp.n_sms = ctx->n_sms / 2;
+        *v_out = 3;
+        *G_out = choose_regions_n(&tmp, n_pairs, tc_ntiles(ctx, 3));
+        return true;
     }
     if (ok1) {
         *v_out = 1;
@@ -759,7 +811,8 @@ dock_status run_grid_tc(dock_ctx* ctx, int m, int n_slots, const float* Lw, floa
     TRY(pack_weights_tc(ctx, m, ctx->tcplan[v][m], n_slots, Lw));
     tc::TcArgs a = tc_args(ctx, m, v, n_slots, G, static_cast<const unsigned char*>(ctx->Wtc.p));
     a.grid = grid;
-    CU(launch_tc<true>(m, v, ctx->tcplan[v][m], a, (int)(n_blocks * G), ctx->stream));
+    const int64_t items = v == 3 ? 2 * ((n_blocks + 1) / 2) * G : n_blocks * G;
+    CU(launch_tc<true>(m, v, ctx->tcplan[v][m], a, (int)items, ctx->stream));
     ctx->kernels_last++;
     return DOCK_OK;
 }
@@ -947,7 +1000,9 @@ dock_status dock_init(const dock_grid_desc* g, const float* receptor, const floa
     for (int m = 1; m <= ctx->m_max; m++) {
         dock_status s = make_plan(ctx, m);
         if (s != DOCK_OK && m == ctx->m_max) return bail(s);
-        if (make_tc_plan(ctx, m, 1) != DOCK_OK || make_tc_plan(ctx, m, 2) != DOCK_OK) return bail(DOCK_E_CUDA);
+        if (make_tc_plan(ctx, m, 1) != DOCK_OK || make_tc_plan(ctx, m, 2) != DOCK_OK ||
+            make_tc_plan(ctx, m, 3) != DOCK_OK)
+            return bail(DOCK_E_CUDA);
     }
     *out = ctx;
     return DOCK_OK;
@@ -967,7 +1022,7 @@ dock_status dock_set_tuning(dock_ctx* ctx, int key, int64_t value)
             ctx->engine = (int)value;
             return DOCK_OK;
         case DOCK_TUNE_TC_VARIANT:
-            if (value < 0 || value > 2) return fail(ctx, DOCK_E_INVALID_ARG, "tc variant must be 0, 1 or 2");
+            if (value < 0 || value > 3) return fail(ctx, DOCK_E_INVALID_ARG, "tc variant must be 0..3");
             ctx->tc_variant = (int)value;
             return DOCK_OK;
         case DOCK_TUNE_TC_EPILOGUE_WARPS:
@@ -1105,7 +1160,7 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
         ta.mu = mup;
         ta.cnt = cntp;
         ta.cand = candp;
-        const int64_t items = n_blocks * G;
+        const int64_t items = v == 3 ? 2 * ((n_blocks + 1) / 2) * G : n_blocks * G;
         if (items > 0x7fffffff) return fail(ctx, DOCK_E_UNSUPPORTED, "too many work items");
         CU(cudaEventRecord(ctx->ev_corr[0], ctx->stream));
         CU(launch_tc<false>(m, v, ctx->tcplan[v][m], ta, (int)items, ctx->stream));

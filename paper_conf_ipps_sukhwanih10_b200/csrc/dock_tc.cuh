@@ -694,4 +694,338 @@ __global__ void k_pack_weights_tc_pair(const float* __restrict__ Lw, unsigned ch
     }
 }
 
+// ------------------------------------------------------------------ variant 3: cta_group::2
+
+__device__ __forceinline__ void umma_bf16_2sm(uint32_t d_tmem, uint64_t a, uint64_t b, uint32_t idesc, uint32_t acc)
+{
+    asm volatile(
+        "{\n\t.reg .pred p;\n\tsetp.ne.b32 p, %4, 0;\n\t"
+        "tcgen05.mma.cta_group::2.kind::f16 [%0], %1, %2, %3, p;\n\t}\n" ::"r"(d_tmem),
+        "l"(a), "l"(b), "r"(idesc), "r"(acc)
+        : "memory");
+}
+__device__ __forceinline__ void umma_commit_2sm_mc(uint64_t* bar, uint16_t mask)
+{
+    asm volatile(
+        "tcgen05.commit.cta_group::2.mbarrier::arrive::one.shared::cluster.multicast::cluster.b64 [%0], %1;" ::"r"(
+            dk::smem_u32(bar)),
+        "h"(mask)
+        : "memory");
+}
+// Arrive on the barrier at the same shared-memory offset in CTA `rank` of the cluster.
+__device__ __forceinline__ void mbar_arrive_remote(uint64_t* bar, uint32_t rank)
+{
+    asm volatile(
+        "{\n\t.reg .b32 ra;\n\tmapa.shared::cluster.u32 ra, %0, %1;\n\t"
+        "mbarrier.arrive.release.cluster.shared::cluster.b64 _, [ra];\n\t}\n" ::"r"(dk::smem_u32(bar)),
+        "r"(rank)
+        : "memory");
+}
+
+// Variant 3: a CTA pair runs 256 rotations (its two blocks) against 4 receptor rows per tile,
+// each CTA holding 2 of the rows.  The leader issues tcgen05.mma.cta_group::2 M = 256 x N = 256:
+// A = each CTA's own 128 rotations, B = CTA0's row q (N 0..127) and CTA1's row q (N 128..255),
+// D = each CTA's TMEM [128 rotations][2 accumulators x 256 columns].  Per SM this halves the
+// shared-memory operand reads and the MMA instructions of variant 1.  Loads complete on local
+// barriers; the peer's MMA warp relays "stage full" to the leader with a remote arrive, and the
+// leader's commits release stages in both CTAs (multicast).
+template <int M, bool GRID>
+__global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc2(const __grid_constant__ CUtensorMap tmap,
+                                                           const __grid_constant__ CUtensorMap tmap_pair, const TcArgs a)
+{
+    constexpr int KS = KSTEPS;
+    constexpr unsigned STAGE = KS * WCHUNK;
+    constexpr int QL = 2;                 // receptor rows per CTA per tile; the pair covers 4
+    constexpr int MXP = (M + 1) / 2, MXQ = (M + 3) / 4;
+    extern __shared__ __align__(1024) unsigned char smem[];
+    __shared__ uint64_t bars[2 * 2 + 2 * WSTAGES + 2 + 2 + WSTAGES];
+    __shared__ uint32_t tmem_base_s;
+    uint64_t* rec_full = bars;
+    uint64_t* rec_empty = bars + 2;
+    uint64_t* w_full = bars + 4;
+    uint64_t* w_empty = w_full + WSTAGES;
+    uint64_t* tm_full = w_empty + WSTAGES;
+    uint64_t* tm_empty = tm_full + 1;
+    uint64_t* peer_rec = tm_empty + 1;    // leader only: peer's receptor buffers landed
+    uint64_t* peer_w = peer_rec + 2;      // leader only: peer's weight stages landed
+
+    uint32_t crank;
+    asm volatile("mov.u32 %0, %%cluster_ctarank;" : "=r"(crank));
+    const bool leader = crank == 0;
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    const int pitem = blockIdx.x >> 1;
+    const int bp = pitem / a.G, region = pitem % a.G;
+    const int block = 2 * bp + static_cast<int>(crank);
+    const int tile_begin = region * a.tiles_per_region;
+    const int tile_end = min(a.ntiles, tile_begin + a.tiles_per_region);
+    const int n_tiles = tile_end - tile_begin;
+    unsigned char* rec_smem = smem;
+    unsigned char* w_smem = smem + 2 * a.rec_stage_bytes;
+
+    if (threadIdx.x == 0) {
+        for (int i = 0; i < 2; i++) {
+            dk::mbar_init(&rec_full[i], 1);
+            dk::mbar_init(&rec_empty[i], 1);
+            dk::mbar_init(&peer_rec[i], 1);
+        }
+        for (int i = 0; i < a.wstages; i++) {
+            dk::mbar_init(&w_full[i], 1);
+            dk::mbar_init(&w_empty[i], 1);
+            dk::mbar_init(&peer_w[i], 1);
+        }
+        dk::mbar_init(&tm_full[0], 1);
+        dk::mbar_init(&tm_empty[0], 2 * a.nepi);
+        dk::fence_mbar_init();
+    }
+    if (warp == 1) {
+        asm volatile("tcgen05.alloc.cta_group::2.sync.aligned.shared::cta.b32 [%0], 512;" ::"r"(
+            dk::smem_u32(&tmem_base_s)));
+        asm volatile("tcgen05.relinquish_alloc_permit.cta_group::2.sync.aligned;");
+    }
+    tc_fence_before();
+    __syncthreads();
+    cluster_sync_all();
+    tc_fence_after();
+    const uint32_t tmem = tmem_base_s;
+
+    if (n_tiles > 0) {
+        if (warp == 0) {
+            // ------------------------------------------------ TMA producer (both CTAs, local data)
+            if (elect_one()) {
+                dk::prefetch_tmap(&tmap);
+                dk::prefetch_tmap(&tmap_pair);
+            }
+            const unsigned char* wsrc = a.W + static_cast<size_t>(block) * a.nsteps * WCHUNK;
+            int ws = 0, wph = 0, wuse = 0;
+            auto stream_weights = [&](int s0, int s1) {
+                for (int s = s0; s < s1; s += KS) {
+                    if (wuse >= a.wstages) dk::mbar_wait(&w_empty[ws], wph ^ 1);
+                    if (elect_one()) {
+                        dk::mbar_arrive_expect_tx(&w_full[ws], STAGE);
+                        dk::bulk_load(w_smem + static_cast<size_t>(ws) * STAGE, wsrc + static_cast<size_t>(s) * WCHUNK,
+                                      STAGE, &w_full[ws]);
+                    }
+                    __syncwarp();
+                    wuse++;
+                    if (++ws == a.wstages) {
+                        ws = 0;
+                        wph ^= 1;
+                    }
+                }
+            };
+            for (int ti = 0; ti < n_tiles; ti++) {
+                const int tile = tile_begin + ti;
+                const int tx = tile % a.ntx, ty = (tile / a.ntx) % a.nty, tz = tile / (a.ntx * a.nty);
+                const int y0 = ty * (2 * QL) + QL * static_cast<int>(crank);
+                if (ti > 0) dk::mbar_wait(&rec_empty[0], (ti - 1) & 1);
+                if (elect_one()) {
+                    dk::mbar_arrive_expect_tx(&rec_full[0], a.box_bytes);
+                    tma_load_5d(rec_smem, &tmap, 0, tx * NT, y0, tz, 0, &rec_full[0]);
+                }
+                __syncwarp();
+                stream_weights(0, a.S1p);
+                if (ti > 0) dk::mbar_wait(&rec_empty[1], (ti - 1) & 1);
+                if (elect_one()) {
+                    dk::mbar_arrive_expect_tx(&rec_full[1], a.box_bytes);
+                    tma_load_5d(rec_smem + a.rec_stage_bytes, &tmap_pair, 0, tx * NT, y0, tz, 0, &rec_full[1]);
+                }
+                __syncwarp();
+                stream_weights(a.S1p, a.nsteps);
+            }
+        } else if (warp == 1) {
+            if (!leader) {
+                // ------------------------------------------------ relay: tell the leader our stages landed
+                int ws = 0, wph = 0;
+                auto relay_stages = [&](int n) {
+                    for (int s = 0; s < n; s += KS) {
+                        dk::mbar_wait(&w_full[ws], wph);
+                        if (elect_one()) mbar_arrive_remote(&peer_w[ws], 0);
+                        __syncwarp();
+                        if (++ws == a.wstages) {
+                            ws = 0;
+                            wph ^= 1;
+                        }
+                    }
+                };
+                for (int ti = 0; ti < n_tiles; ti++) {
+                    dk::mbar_wait(&rec_full[0], ti & 1);
+                    if (elect_one()) mbar_arrive_remote(&peer_rec[0], 0);
+                    __syncwarp();
+                    relay_stages(a.S1p);
+                    dk::mbar_wait(&rec_full[1], ti & 1);
+                    if (elect_one()) mbar_arrive_remote(&peer_rec[1], 0);
+                    __syncwarp();
+                    relay_stages(a.S2p);
+                }
+            } else {
+                // ------------------------------------------------ leader: MMA issue for the pair
+                constexpr uint32_t idesc = umma_idesc(2 * ROT, 2 * NT);
+                constexpr uint16_t PAIRMASK = 3;
+                const uint32_t rec0 = dk::smem_u32(rec_smem), w0 = dk::smem_u32(w_smem);
+                const uint64_t dA0 = umma_desc(w0, ROT * 16, 128);
+                const uint64_t dB0 = umma_desc(rec0, 16, 128);
+                const uint64_t dP0 = umma_desc(rec0 + a.rec_stage_bytes, 32, 128);
+                const uint32_t row16 = static_cast<uint32_t>(a.TXB) * 16u;
+                const uint32_t rowTY = static_cast<uint32_t>(a.TYB) * row16;
+                int ws = 0, wph = 0;
+                auto issue_stage = [&](int kind, int s0, bool first) {
+                    dk::mbar_wait(&w_full[ws], wph);
+                    dk::mbar_wait(&peer_w[ws], wph);
+                    tc_fence_after();
+                    if (elect_one()) {
+                        const uint64_t da0 = dA0 + ((static_cast<uint32_t>(ws) * STAGE) >> 4);
+#pragma unroll
+                        for (int ks = 0; ks < KS; ks++) {
+                            const int s = s0 + ks;
+                            uint64_t db;
+                            if (kind == 0) {
+                                const int vxp = s % MXP, vy = (s / MXP) % M, vz = s / (MXP * M);
+                                db = s < a.S1 ? dB0 + ((vz * rowTY + vy * row16 + vxp * 32u) >> 4) : dB0;
+                            } else {
+                                const int vxq = s % MXQ, vy = (s / MXQ) % M, vz = s / (MXQ * M);
+                                db = s < a.S2 ? dP0 + ((vz * rowTY + vy * row16 + vxq * 64u) >> 4) : dP0;
+                            }
+                            const uint64_t da = da0 + ((ks * WCHUNK) >> 4);
+#pragma unroll
+                            for (int q = 0; q < QL; q++)
+                                umma_bf16_2sm(tmem + q * 2 * NT, da, db + ((q * row16) >> 4), idesc,
+                                              (first && ks == 0) ? 0u : 1u);
+                        }
+                        umma_commit_2sm_mc(&w_empty[ws], PAIRMASK);
+                    }
+                    __syncwarp();
+                    if (++ws == a.wstages) {
+                        ws = 0;
+                        wph ^= 1;
+                    }
+                };
+                for (int ti = 0; ti < n_tiles; ti++) {
+                    dk::mbar_wait(&rec_full[0], ti & 1);
+                    dk::mbar_wait(&peer_rec[0], ti & 1);
+                    if (ti > 0) dk::mbar_wait(&tm_empty[0], (ti - 1) & 1);
+                    tc_fence_after();
+                    for (int s = 0; s < a.S1p; s += KS) issue_stage(0, s, s == 0);
+                    if (elect_one()) umma_commit_2sm_mc(&rec_empty[0], PAIRMASK);
+                    __syncwarp();
+                    dk::mbar_wait(&rec_full[1], ti & 1);
+                    dk::mbar_wait(&peer_rec[1], ti & 1);
+                    tc_fence_after();
+                    for (int s = 0; s < a.S2p; s += KS) issue_stage(1, s, false);
+                    if (elect_one()) {
+                        umma_commit_2sm_mc(&rec_empty[1], PAIRMASK);
+                        umma_commit_2sm_mc(&tm_full[0], PAIRMASK);
+                    }
+                    __syncwarp();
+                }
+            }
+        } else if (warp < 2 + a.nepi) {
+            // ------------------------------------------------ epilogue warps (both CTAs)
+            const int quarter = warp & 3;
+            const int cls = (warp - 2) >> 2;                 // 0..3 -> (accumulator q, CTA half)
+            const int nclass = a.nepi >> 2;
+            const int r = quarter * 32 + lane;
+            const int slot = block * ROT + r;
+            const bool rot_ok = slot < a.n_slots;
+            unsigned long long lst[LIST];
+#pragma unroll
+            for (int i = 0; i < LIST; i++) lst[i] = KEY_MAX;
+            float th = __int_as_float(0x7f800000);
+            uint32_t th_t = 0xffffffffu;
+            for (int ti = 0; ti < n_tiles; ti++) {
+                const int tile = tile_begin + ti;
+                dk::mbar_wait(&tm_full[0], ti & 1);
+                tc_fence_after();
+                const int tx = tile % a.ntx, ty = (tile / a.ntx) % a.nty, tz = tile / (a.ntx * a.nty);
+                for (int c4 = cls; c4 < 4; c4 += nclass) {
+                    const int q = c4 >> 1, half = c4 & 1;
+                    const int y = ty * (2 * QL) + QL * half + q, z = tz;
+                    const bool row_ok = rot_ok && y < a.ny && z < a.nz;
+                    const int x0 = tx * NT;
+                    const uint32_t tbase = static_cast<uint32_t>((z * a.ny + y) * a.nx + x0);
+#pragma unroll 1
+                    for (int c0 = 0; c0 < NT; c0 += 32) {
+                        uint32_t v[32];
+                        tmem_ld32(tmem + (static_cast<uint32_t>(quarter * 32) << 16) + q * 2 * NT + half * NT + c0, v);
+                        if (!row_ok) continue;
+                        if constexpr (GRID) {
+                            float* out = a.grid + static_cast<size_t>(slot) * a.nx * a.ny * a.nz + tbase;
+#pragma unroll
+                            for (int j = 0; j < 32; j++)
+                                if (x0 + c0 + j < a.nx) out[c0 + j] = __uint_as_float(v[j]);
+                        } else {
+                            float mn = __uint_as_float(v[0]);
+#pragma unroll
+                            for (int j = 1; j < 32; j++) mn = fminf(mn, __uint_as_float(v[j]));
+                            if (mn < th || (mn == th && tbase + c0 < th_t)) {
+                                const int jmax = min(32, a.nx - x0 - c0);
+                                uint32_t msk = 0;
+#pragma unroll
+                                for (int j = 0; j < 32; j++)
+                                    msk |= (__uint_as_float(v[j]) <= th && j < jmax) ? (1u << j) : 0u;
+                                while (msk) {
+                                    const int j = __ffs(msk) - 1;
+                                    msk &= msk - 1;
+                                    const float sv = __uint_as_float(select32(v, j));
+                                    if (sv <= th) {
+                                        const unsigned long long key = dk::make_key(sv, tbase + c0 + j);
+                                        if (key < lst[LIST - 1]) {
+                                            list_insert(lst, key);
+                                            th = dk::key_score_bound(static_cast<uint32_t>(lst[LIST - 1] >> 32));
+                                            th_t = static_cast<uint32_t>(lst[LIST - 1] & 0xffffffffu);
+                                        }
+                                    }
+                                }
+                            }
+                        }
+                    }
+                }
+                tc_fence_before();
+                __syncwarp();
+                if (lane == 0) {
+                    if (leader) dk::mbar_arrive(&tm_empty[0]);
+                    else mbar_arrive_remote(&tm_empty[0], 0);
+                }
+            }
+            if constexpr (!GRID) {
+                if (rot_ok) {
+                    unsigned long long Tw = KEY_MAX;
+                    uint32_t chosen[32];
+                    int nc = 0;
+#pragma unroll
+                    for (int i = 0; i < LIST; i++) {
+                        const unsigned long long key = lst[i];
+                        if (key != KEY_MAX && nc < a.k) {
+                            const uint32_t t = static_cast<uint32_t>(key & 0xffffffffu);
+                            bool far = true;
+                            for (int c = 0; c < nc; c++)
+                                far = far && dk::cheb_cyc(t, chosen[c], a.nx, a.ny, a.nz) > 2 * a.rho;
+                            if (far) {
+                                chosen[nc] = t;
+                                nc++;
+                                if (nc == a.k) Tw = key;
+                            }
+                        }
+                    }
+                    const unsigned long long old = atomicMin(&a.T[slot], Tw);
+                    const unsigned long long Tn = old < Tw ? old : Tw;
+                    atomicMin(&a.mu[slot], lst[LIST - 1]);
+#pragma unroll
+                    for (int i = 0; i < LIST; i++) {
+                        const unsigned long long key = lst[i];
+                        if (key != KEY_MAX && key <= Tn) {
+                            const unsigned pos = atomicAdd(&a.cnt[slot], 1u);
+                            if (pos < static_cast<unsigned>(a.cap)) a.cand[static_cast<size_t>(slot) * a.cap + pos] = key;
+                        }
+                    }
+                }
+            }
+        }
+    }
+    tc_fence_before();
+    __syncthreads();
+    cluster_sync_all();
+    if (warp == 1) asm volatile("tcgen05.dealloc.cta_group::2.sync.aligned.b32 %0, 512;" ::"r"(tmem));
+    cluster_sync_all();
+}
+
 }  // namespace tc
