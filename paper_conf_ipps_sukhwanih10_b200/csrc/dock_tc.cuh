@@ -273,23 +273,44 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                 }
             };
             if constexpr (PAIR) {
-                for (int ti = 0; ti < n_tiles; ti++) {
-                    const int tile = tile_begin + ti;
+                // Receptor boxes are issued as soon as their buffer frees: the producer polls the
+                // release barriers between weight stages (main(t+1) needs pass 1 of t done, pair(t+1)
+                // pass 2 of t), and blocks only right before the first stage that needs a box.
+                int pm = 0, pp = 0;   // next main / pair box (tile index) to load
+                auto issue_box = [&](int which, int t) {
+                    const int tile = tile_begin + t;
                     const int tx = tile % a.ntx, ty = (tile / a.ntx) % a.nty, tz = tile / (a.ntx * a.nty);
-                    if (ti > 0) dk::mbar_wait(&rec_empty[0], (ti - 1) & 1);
                     if (elect_one()) {
-                        dk::mbar_arrive_expect_tx(&rec_full[0], a.box_bytes);
-                        tma_load_5d(rec_smem, &tmap, 0, tx * NT, ty * Q, tz, 0, &rec_full[0]);
+                        dk::mbar_arrive_expect_tx(&rec_full[which], a.box_bytes);
+                        tma_load_5d(rec_smem + which * a.rec_stage_bytes, which ? &tmap_pair : &tmap, 0, tx * NT,
+                                    ty * Q, tz, 0, &rec_full[which]);
                     }
                     __syncwarp();
-                    stream_weights(0, a.S1p);
-                    if (ti > 0) dk::mbar_wait(&rec_empty[1], (ti - 1) & 1);
-                    if (elect_one()) {
-                        dk::mbar_arrive_expect_tx(&rec_full[1], a.box_bytes);
-                        tma_load_5d(rec_smem + a.rec_stage_bytes, &tmap_pair, 0, tx * NT, ty * Q, tz, 0, &rec_full[1]);
+                };
+                auto poll = [&](int ti) {
+                    if (pm < n_tiles && pm <= ti + 1 && (pm == 0 || dk::mbar_test(&rec_empty[0], (pm - 1) & 1)))
+                        issue_box(0, pm++);
+                    if (pp < n_tiles && pp <= ti + 1 && (pp == 0 || dk::mbar_test(&rec_empty[1], (pp - 1) & 1)))
+                        issue_box(1, pp++);
+                };
+                auto ensure = [&](int which, int t) {
+                    int& nx = which ? pp : pm;
+                    if (nx == t) {
+                        if (t > 0) dk::mbar_wait(&rec_empty[which], (t - 1) & 1);
+                        issue_box(which, nx++);
                     }
-                    __syncwarp();
-                    stream_weights(a.S1p, a.nsteps);
+                };
+                for (int ti = 0; ti < n_tiles; ti++) {
+                    ensure(0, ti);
+                    for (int s = 0; s < a.S1p; s += KS) {
+                        poll(ti);
+                        stream_weights(s, s + KS);
+                    }
+                    ensure(1, ti);
+                    for (int s = a.S1p; s < a.nsteps; s += KS) {
+                        poll(ti);
+                        stream_weights(s, s + KS);
+                    }
                 }
             } else {
             for (int ti = 0; ti < n_tiles; ti++) {
@@ -813,24 +834,42 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc2(const __grid_constant_
                     }
                 }
             };
-            for (int ti = 0; ti < n_tiles; ti++) {
-                const int tile = tile_begin + ti;
+            int pm = 0, pp = 0;
+            auto issue_box = [&](int which, int t) {
+                const int tile = tile_begin + t;
                 const int tx = tile % a.ntx, ty = (tile / a.ntx) % a.nty, tz = tile / (a.ntx * a.nty);
                 const int y0 = ty * (2 * QL) + QL * static_cast<int>(crank);
-                if (ti > 0) dk::mbar_wait(&rec_empty[0], (ti - 1) & 1);
                 if (elect_one()) {
-                    dk::mbar_arrive_expect_tx(&rec_full[0], a.box_bytes);
-                    tma_load_5d(rec_smem, &tmap, 0, tx * NT, y0, tz, 0, &rec_full[0]);
+                    dk::mbar_arrive_expect_tx(&rec_full[which], a.box_bytes);
+                    tma_load_5d(rec_smem + which * a.rec_stage_bytes, which ? &tmap_pair : &tmap, 0, tx * NT, y0, tz,
+                                0, &rec_full[which]);
                 }
                 __syncwarp();
-                stream_weights(0, a.S1p);
-                if (ti > 0) dk::mbar_wait(&rec_empty[1], (ti - 1) & 1);
-                if (elect_one()) {
-                    dk::mbar_arrive_expect_tx(&rec_full[1], a.box_bytes);
-                    tma_load_5d(rec_smem + a.rec_stage_bytes, &tmap_pair, 0, tx * NT, y0, tz, 0, &rec_full[1]);
+            };
+            auto poll = [&](int ti) {
+                if (pm < n_tiles && pm <= ti + 1 && (pm == 0 || dk::mbar_test(&rec_empty[0], (pm - 1) & 1)))
+                    issue_box(0, pm++);
+                if (pp < n_tiles && pp <= ti + 1 && (pp == 0 || dk::mbar_test(&rec_empty[1], (pp - 1) & 1)))
+                    issue_box(1, pp++);
+            };
+            auto ensure = [&](int which, int t) {
+                int& nx = which ? pp : pm;
+                if (nx == t) {
+                    if (t > 0) dk::mbar_wait(&rec_empty[which], (t - 1) & 1);
+                    issue_box(which, nx++);
                 }
-                __syncwarp();
-                stream_weights(a.S1p, a.nsteps);
+            };
+            for (int ti = 0; ti < n_tiles; ti++) {
+                ensure(0, ti);
+                for (int s = 0; s < a.S1p; s += KS) {
+                    poll(ti);
+                    stream_weights(s, s + KS);
+                }
+                ensure(1, ti);
+                for (int s = a.S1p; s < a.nsteps; s += KS) {
+                    poll(ti);
+                    stream_weights(s, s + KS);
+                }
             }
         } else if (warp == 1) {
             if (!leader) {
