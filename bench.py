@@ -52,7 +52,7 @@ def parse():
                     help="correlation engine: auto (tcgen05 when eligible), ffma (FP32 FFMA), tc (tcgen05 bf16x3)")
     ap.add_argument("--no-alt", action="store_true", help="skip the secondary measurement of the other engine")
     ap.add_argument("--tc-epi", type=int, default=0, choices=[0, 4, 8, 16], help="tcgen05 epilogue warps (0 auto)")
-    ap.add_argument("--tc-variant", type=int, default=0, choices=[0, 1, 2, 3],
+    ap.add_argument("--tc-variant", type=int, default=0, choices=[0, 1, 2, 3, 4],
                     help="tcgen05 tiling: 0 auto, 1 = 4 rows x 1 TMEM buffer, 2 = CTA pair, 2 rows x 2 buffers")
     return ap.parse_args()
 
@@ -201,7 +201,7 @@ def roofline(pk, pk_kind, info, c, flops_launch, corr_ms, ms_step, units_local):
         executed = flops_launch * (ks * 16.0) / (c.P * c.m ** 3)
         v = int(info.get("tc_variant_last", 1)) or 1
         kname = {1: f"k_corr_tc<{c.m},4,1,1,PAIR,false>", 2: f"k_corr_tc<{c.m},2,2,2,PAIR,false>",
-                 3: f"k_corr_tc2<{c.m},false>"}.get(v, "k_corr_tc")
+                 3: f"k_corr_tc2<{c.m},false>", 4: f"k_corr_tc<{c.m},2,2,1,PAIR,false>"}.get(v, "k_corr_tc")
         return {"bound": "tensor", "engine": f"tcgen05 bf16x3 (variant {v})", "kernel": kname,
                 "achieved": achieved, "peak": peak, "unit": "TFLOP/s", "frac": achieved / peak, "traffic": None,
                 "peak_source": f"bf16 dense tensor peak, burst, MEASURED_PEAKS.json ({pk_kind})",

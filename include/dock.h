@@ -138,7 +138,7 @@ typedef enum {
     DOCK_TUNE_ENGINE = 4,         /* correlation engine: 0 auto (tcgen05 when eligible), 1 FP32 FFMA, 2 tcgen05 */
     DOCK_TUNE_TC_VARIANT = 5,     /* tcgen05 tiling: 0 auto, 1 = 4 rows x 1 TMEM buffer, 2 = 2 rows x 2 buffers on a
                                      CTA pair with multicast weight streaming, 3 = cta_group::2 (M = 256 rotations,
-                                     N = 256 translations over a CTA pair) */
+                                     N = 256 translations over a CTA pair), 4 = 2 rows x 2 TMEM buffers, single CTA */
     DOCK_TUNE_TC_EPILOGUE_WARPS = 6 /* tcgen05 epilogue warps: 0 auto (one translation row per thread), 4, 8, 16 */
 } dock_tune_key;
 

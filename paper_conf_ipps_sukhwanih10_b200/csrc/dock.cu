@@ -74,7 +74,7 @@ struct dock_ctx {
     uint16_t* d_rec_tc = nullptr;
     uint16_t* d_rec_pair = nullptr;   // PAIR-scheme receptor copy (P <= 4)
     int tc_Gch = 0, tc_ntx = 0, tc_ntz = 0, tc_Xp = 0, tc_Yp = 0, tc_Zp = 0;
-    TcPlan tcplan[4][DOCK_MAX_M + 1];   // [variant][m]
+    TcPlan tcplan[5][DOCK_MAX_M + 1];   // [variant][m]
     DevBuf Wtc;
     // per-call scratch (grow-only)
     DevBuf xyz, coef, off, rot, Lw, T, mu, cnt, cand, poses, fb_list, grid, slots, units, Lw_fb, picks;
@@ -274,9 +274,9 @@ cudaError_t launch_corr(int m, const MPlan& pl, const dk::CorrArgs& a, int grid,
 
 int tc_txb(int m) { return tc::NT + (m + 1) / 2 * 2 - 1; }
 // tcgen05 variants: 1 = Q4 rows x 1 TMEM buffer, single CTA; 2 = Q2 rows x 2 buffers, CTA pair + multicast.
-// tile rows (translation rows per tile): variants 1 and 3 tile 4 rows, variant 2 tiles 2
-inline int tc_q(int v) { return v == 2 ? 2 : 4; }
-inline int tc_cl(int v) { return v == 1 ? 1 : 2; }
+// tile rows (translation rows per tile): variants 1 and 3 tile 4 rows, variants 2 and 4 tile 2
+inline int tc_q(int v) { return (v == 2 || v == 4) ? 2 : 4; }
+inline int tc_cl(int v) { return (v == 1 || v == 4) ? 1 : 2; }
 // receptor rows held per CTA (variant 3 splits the 4 tile rows over the CTA pair)
 inline int tc_rows_cta(int v) { return v == 1 ? 4 : 2; }
 inline int tc_nty(const dock_ctx* c, int v) { return (c->ny + tc_q(v) - 1) / tc_q(v); }
@@ -367,7 +367,7 @@ cudaError_t launch_tc_t(const TcPlan& pl, const tc::TcArgs& a, int grid, cudaStr
 template <int V, bool PAIR, bool GRID>
 cudaError_t launch_tc_v(int m, const TcPlan& pl, const tc::TcArgs& a, int grid, cudaStream_t st)
 {
-    constexpr int Q = V == 1 ? 4 : 2, NB = V == 1 ? 1 : 2, CL = V == 1 ? 1 : 2;
+    constexpr int Q = V == 1 ? 4 : 2, NB = V == 1 ? 1 : 2, CL = (V == 1 || V == 4) ? 1 : 2;
     switch (m) {
         case 1: return launch_tc_t<1, Q, NB, CL, PAIR, GRID>(pl, a, grid, st);
         case 2: return launch_tc_t<2, Q, NB, CL, PAIR, GRID>(pl, a, grid, st);
@@ -425,6 +425,7 @@ cudaError_t launch_tc(int m, int v, const TcPlan& pl, const tc::TcArgs& a, int g
 {
     if (v == 3) return launch_tc2<GRID>(m, pl, a, grid, st);
     if (!pl.pair) return v == 1 ? launch_tc_v<1, false, GRID>(m, pl, a, grid, st) : cudaErrorInvalidValue;
+    if (v == 4) return launch_tc_v<4, true, GRID>(m, pl, a, grid, st);
     return v == 1 ? launch_tc_v<1, true, GRID>(m, pl, a, grid, st) : launch_tc_v<2, true, GRID>(m, pl, a, grid, st);
 }
 
@@ -732,7 +733,7 @@ tc::TcArgs tc_args(dock_ctx* ctx, int m, int v, int n_slots, int G, const unsign
     a.rec_stage_bytes = tp.rec_stage_bytes;
     a.n_rec_stages = tp.n_rec_stages;
     a.wstages = tp.wstages;
-    a.nepi = ctx->tc_nepi > 0 ? std::min(16, ctx->tc_nepi) : (v == 2 ? 8 : 16);   // one row per thread
+    a.nepi = ctx->tc_nepi > 0 ? std::min(16, ctx->tc_nepi) : ((v == 2 || v == 4) ? 8 : 16);   // one row per thread
     a.S1 = tp.S1;
     a.S1p = tp.S1p;
     a.S2 = tp.S2;
@@ -754,6 +755,11 @@ bool plan_tc_launch(dock_ctx* ctx, int m, int n_slots, int* v_out, int* G_out)
             *G_out = G;
             return true;
         }
+    }
+    if (ctx->tc_variant == 4 && ctx->tcplan[4][m].ok) {
+        *v_out = 4;
+        *G_out = choose_regions_n(ctx, n_blocks, tc_ntiles(ctx, 4));
+        return true;
     }
     if (ctx->tc_variant == 3 && ctx->tcplan[3][m].ok) {
         // CTA pairs over pairs of rotation blocks; a pair occupies two SMs
@@ -1001,7 +1007,7 @@ dock_status dock_init(const dock_grid_desc* g, const float* receptor, const floa
         dock_status s = make_plan(ctx, m);
         if (s != DOCK_OK && m == ctx->m_max) return bail(s);
         if (make_tc_plan(ctx, m, 1) != DOCK_OK || make_tc_plan(ctx, m, 2) != DOCK_OK ||
-            make_tc_plan(ctx, m, 3) != DOCK_OK)
+            make_tc_plan(ctx, m, 3) != DOCK_OK || make_tc_plan(ctx, m, 4) != DOCK_OK)
             return bail(DOCK_E_CUDA);
     }
     *out = ctx;
@@ -1022,7 +1028,7 @@ dock_status dock_set_tuning(dock_ctx* ctx, int key, int64_t value)
             ctx->engine = (int)value;
             return DOCK_OK;
         case DOCK_TUNE_TC_VARIANT:
-            if (value < 0 || value > 3) return fail(ctx, DOCK_E_INVALID_ARG, "tc variant must be 0..3");
+            if (value < 0 || value > 4) return fail(ctx, DOCK_E_INVALID_ARG, "tc variant must be 0..4");
             ctx->tc_variant = (int)value;
             return DOCK_OK;
         case DOCK_TUNE_TC_EPILOGUE_WARPS:
