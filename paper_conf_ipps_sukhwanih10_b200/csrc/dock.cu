@@ -12,6 +12,7 @@
 #include <cmath>
 #include <cstdarg>
 #include <cstdio>
+#include <cstdlib>
 #include <cstring>
 #include <new>
 #include <vector>
@@ -76,6 +77,10 @@ struct dock_ctx {
     int tc_Gch = 0, tc_ntx = 0, tc_ntz = 0, tc_Xp = 0, tc_Yp = 0, tc_Zp = 0;
     TcPlan tcplan[5][DOCK_MAX_M + 1];   // [variant][m]
     DevBuf Wtc;
+    // diagnostics (environment, read at init): DOCK_TC_TRACE=1 prints per-role cycle counters of every
+    // k_corr_tc launch to stderr; DOCK_TC_DEBUG=1|2 disables parts of the epilogue (timing only)
+    unsigned long long* d_trace = nullptr;
+    int tc_dbg = 0;
     // per-call scratch (grow-only)
     DevBuf xyz, coef, off, rot, Lw, T, mu, cnt, cand, poses, fb_list, grid, slots, units, Lw_fb, picks;
     int* d_small = nullptr;    // [0] status, [1] fb_cnt, [2] cand_max
@@ -300,6 +305,9 @@ dock_status make_tc_plan(dock_ctx* ctx, int m, int v)
     pl.TYB = tc_rows_cta(v) + m - 1;
     pl.TZB = m;
     pl.box_bytes = 16 * pl.TXB * pl.TYB * pl.TZB;
+    // the single-CTA PAIR kernels bake the box geometry into their descriptor offsets
+    if (pl.pair && tc_cl(v) == 1 && (pl.TXB != tc::pair_txb(m) || pl.TYB != tc_q(v) + m - 1))
+        return fail(ctx, DOCK_E_CUDA, "tcgen05 PAIR box geometry mismatch");
     pl.rec_stage_bytes = round_up(ctx->tc_Gch * pl.box_bytes, 1024);
     if (pl.pair) {
         pl.S1 = m * m * ((m + 1) / 2);
@@ -734,6 +742,8 @@ tc::TcArgs tc_args(dock_ctx* ctx, int m, int v, int n_slots, int G, const unsign
     a.n_rec_stages = tp.n_rec_stages;
     a.wstages = tp.wstages;
     a.nepi = ctx->tc_nepi > 0 ? std::min(16, ctx->tc_nepi) : ((v == 2 || v == 4) ? 8 : 16);   // one row per thread
+    a.trace = ctx->d_trace;
+    a.dbg = ctx->tc_dbg;
     a.S1 = tp.S1;
     a.S1p = tp.S1p;
     a.S2 = tp.S2;
@@ -854,6 +864,7 @@ void dock_destroy(dock_ctx* ctx)
                       &ctx->cand, &ctx->poses, &ctx->fb_list, &ctx->grid, &ctx->slots, &ctx->units, &ctx->Lw_fb, &ctx->picks};
     for (DevBuf* b : bufs)
         if (b->p) cudaFree(b->p);
+    if (ctx->d_trace) cudaFree(ctx->d_trace);
     if (ctx->d_rec) cudaFree(ctx->d_rec);
     if (ctx->d_rec_tc) cudaFree(ctx->d_rec_tc);
     if (ctx->d_rec_pair) cudaFree(ctx->d_rec_pair);
@@ -907,6 +918,11 @@ dock_status dock_init(const dock_grid_desc* g, const float* receptor, const floa
     }
     if (cudaEventCreate(&ctx->ev_corr[0]) != cudaSuccess || cudaEventCreate(&ctx->ev_corr[1]) != cudaSuccess)
         return bail(DOCK_E_CUDA);
+    if (const char* e = getenv("DOCK_TC_DEBUG")) ctx->tc_dbg = atoi(e);
+    if (const char* e = getenv("DOCK_TC_TRACE")) {
+        if (atoi(e) > 0 && cudaMalloc(&ctx->d_trace, sizeof(unsigned long long) * tc::TR_N) != cudaSuccess)
+            return bail(DOCK_E_OOM);
+    }
     int v = 0;
     if (cudaDeviceGetAttribute(&v, cudaDevAttrMultiProcessorCount, ctx->device) == cudaSuccess) ctx->n_sms = v;
     if (cudaDeviceGetAttribute(&v, cudaDevAttrL2CacheSize, ctx->device) == cudaSuccess) ctx->l2_bytes = v;
@@ -1168,9 +1184,27 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
         ta.cand = candp;
         const int64_t items = v == 3 ? 2 * ((n_blocks + 1) / 2) * G : n_blocks * G;
         if (items > 0x7fffffff) return fail(ctx, DOCK_E_UNSUPPORTED, "too many work items");
+        if (ctx->d_trace) CU(cudaMemsetAsync(ctx->d_trace, 0, sizeof(unsigned long long) * tc::TR_N, ctx->stream));
         CU(cudaEventRecord(ctx->ev_corr[0], ctx->stream));
         CU(launch_tc<false>(m, v, ctx->tcplan[v][m], ta, (int)items, ctx->stream));
         CU(cudaEventRecord(ctx->ev_corr[1], ctx->stream));
+        if (ctx->d_trace) {
+            unsigned long long h[tc::TR_N];
+            CU(cudaMemcpyAsync(h, ctx->d_trace, sizeof(h), cudaMemcpyDeviceToHost, ctx->stream));
+            CU(cudaStreamSynchronize(ctx->stream));
+            const double c = h[tc::TR_CTAS] ? double(h[tc::TR_CTAS]) : 1.0;
+            const double e = h[tc::TR_EPI_WARPS] ? double(h[tc::TR_EPI_WARPS]) : 1.0;
+            fprintf(stderr,
+                    "TCTRACE {\"variant\": %d, \"dbg\": %d, \"ctas\": %llu, \"tiles_per_cta\": %.1f, "
+                    "\"mma_total\": %.0f, \"mma_wait_tmem_empty\": %.0f, \"mma_wait_w_full\": %.0f, "
+                    "\"mma_wait_rec_full\": %.0f, \"epi_total\": %.0f, \"epi_wait_tm_full\": %.0f, "
+                    "\"epi_ldtm\": %.0f, \"prod_total\": %.0f, \"prod_wait_w_empty\": %.0f, "
+                    "\"prod_wait_rec_empty\": %.0f}\n",
+                    v, ctx->tc_dbg, h[tc::TR_CTAS], h[tc::TR_TILES] / c, h[tc::TR_MMA_TOTAL] / c,
+                    h[tc::TR_MMA_TMEMPTY] / c, h[tc::TR_MMA_WFULL] / c, h[tc::TR_MMA_RFULL] / c,
+                    h[tc::TR_EPI_TOTAL] / e, h[tc::TR_EPI_TMFULL] / e, h[tc::TR_EPI_LDTM] / e,
+                    h[tc::TR_PROD_TOTAL] / c, h[tc::TR_PROD_WEMPTY] / c, h[tc::TR_PROD_REMPTY] / c);
+        }
         ctx->regions_last = G;
         ctx->items_last = items;
     } else {

@@ -58,7 +58,28 @@ struct TcArgs {
     unsigned long long* cand;
     // grid mode
     float* grid;
+    // diagnostics (DOCK_TC_TRACE / DOCK_TC_DEBUG environment variables; off on the product path):
+    // trace = per-role cycle counters summed over CTAs (see TR_*); dbg 1 = epilogue skips the TMEM
+    // drain, 2 = drain without candidate processing (timing experiments only: poses are invalid)
+    unsigned long long* trace;
+    int dbg;
 };
+
+// trace counters (cycles summed over CTAs)
+enum { TR_CTAS = 0, TR_TILES, TR_MMA_TOTAL, TR_MMA_TMEMPTY, TR_MMA_WFULL, TR_MMA_RFULL, TR_EPI_TOTAL, TR_EPI_TMFULL,
+       TR_EPI_LDTM, TR_PROD_TOTAL, TR_PROD_WEMPTY, TR_PROD_REMPTY, TR_EPI_WARPS, TR_N = 16 };
+
+// mbarrier wait that adds its duration to `acc` when tracing
+__device__ __forceinline__ void twait(uint64_t* bar, unsigned parity, bool tr, long long& acc)
+{
+    if (tr) {
+        const long long t0 = clock64();
+        dk::mbar_wait(bar, parity);
+        acc += clock64() - t0;
+    } else {
+        dk::mbar_wait(bar, parity);
+    }
+}
 
 __device__ __forceinline__ uint64_t umma_desc(uint32_t saddr, uint32_t lbo, uint32_t sbo)
 {
@@ -176,6 +197,29 @@ __device__ __forceinline__ void umma_commit_mc(uint64_t* bar, uint16_t mask)
         : "memory");
 }
 
+// Shared-memory box geometry of the PAIR scheme (must match make_tc_plan): x extent, y extent.
+__host__ __device__ constexpr int pair_txb(int m)
+{
+    return (128 + (m + 1) / 2 * 2 - 1) > (4 * ((m + 3) / 4) + 126) ? (128 + (m + 1) / 2 * 2 - 1)
+                                                                     : (4 * ((m + 3) / 4) + 126);
+}
+// Byte offset of K-step s inside the PAIR pass-1 box ((hi,lo) voxels, 2 per K-step) and pass-2 box
+// ((hi(x),hi(x+1)) slots, 4 voxels per K-step); padding steps (zero weights) read the box origin.
+__host__ __device__ constexpr uint32_t pair_off1(int m, int s, uint32_t row16, uint32_t rowTY)
+{
+    return s >= m * m * ((m + 1) / 2) ? 0u
+                                      : static_cast<uint32_t>(s / (((m + 1) / 2) * m)) * rowTY +
+                                            static_cast<uint32_t>((s / ((m + 1) / 2)) % m) * row16 +
+                                            static_cast<uint32_t>(s % ((m + 1) / 2)) * 32u;
+}
+__host__ __device__ constexpr uint32_t pair_off2(int m, int s, uint32_t row16, uint32_t rowTY)
+{
+    return s >= m * m * ((m + 3) / 4) ? 0u
+                                      : static_cast<uint32_t>(s / (((m + 3) / 4) * m)) * rowTY +
+                                            static_cast<uint32_t>((s / ((m + 3) / 4)) % m) * row16 +
+                                            static_cast<uint32_t>(s % ((m + 3) / 4)) * 64u;
+}
+
 // CL = 1: one CTA per item.  CL = 2: a cluster of two CTAs works on the same rotation block
 // (two regions with the same number of tiles); each CTA's producer fetches half of every
 // weight chunk and multicasts it into both CTAs' rings, and each MMA warp releases a ring
@@ -193,14 +237,14 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
     static_assert(Q * NBUF * NT <= 512, "TMEM has 512 columns");
     constexpr int MXP = (M + 1) / 2;   // voxel pairs along x (K = 16 = 2 voxels x 8 channels)
     extern __shared__ __align__(1024) unsigned char smem[];
-    __shared__ uint64_t bars[2 * 2 + 2 * WSTAGES + 2 * NBUF];
+    __shared__ uint64_t bars[2 * 2 + 2 * WSTAGES + NBUF + NBUF * Q];
     __shared__ uint32_t tmem_base_s;
     uint64_t* rec_full = bars;
     uint64_t* rec_empty = bars + 2;
     uint64_t* w_full = bars + 4;
     uint64_t* w_empty = w_full + WSTAGES;
     uint64_t* tm_full = w_empty + WSTAGES;
-    uint64_t* tm_empty = tm_full + NBUF;
+    uint64_t* tm_empty = tm_full + NBUF;   // [NBUF][Q]: per accumulator row, so the next tile restarts row by row
 
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     const int block = blockIdx.x / a.G, region = blockIdx.x % a.G;
@@ -219,10 +263,8 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
             dk::mbar_init(&w_full[i], 1);
             dk::mbar_init(&w_empty[i], CL);
         }
-        for (int i = 0; i < NBUF; i++) {
-            dk::mbar_init(&tm_full[i], 1);
-            dk::mbar_init(&tm_empty[i], a.nepi);
-        }
+        for (int i = 0; i < NBUF; i++) dk::mbar_init(&tm_full[i], 1);
+        for (int i = 0; i < NBUF * Q; i++) dk::mbar_init(&tm_empty[i], a.nepi);
         dk::fence_mbar_init();
     }
     if (warp == 1) {
@@ -239,6 +281,8 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
     if constexpr (CL > 1) asm volatile("mov.u32 %0, %%cluster_ctarank;" : "=r"(crank));
     constexpr uint16_t CMASK = (1u << CL) - 1u;
 
+    const bool tr = a.trace != nullptr;
+    long long tw0 = 0, tw1 = 0, tw2 = 0, tstart = tr ? clock64() : 0;   // per-role trace accumulators
     if (n_tiles > 0) {
         if (warp == 0) {
             // ------------------------------------------------ TMA producer (warp-converged, one elected lane)
@@ -251,7 +295,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
             int wuse = 0;
             auto stream_weights = [&](int s0, int s1) {
                 for (int s = s0; s < s1; s += KS) {
-                    if (wuse >= a.wstages) dk::mbar_wait(&w_empty[ws], wph ^ 1);
+                    if (wuse >= a.wstages) twait(&w_empty[ws], wph ^ 1, tr, tw0);
                     if (elect_one()) {
                         dk::mbar_arrive_expect_tx(&w_full[ws], STAGE);
                         if constexpr (CL == 1) {
@@ -296,7 +340,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                 auto ensure = [&](int which, int t) {
                     int& nx = which ? pp : pm;
                     if (nx == t) {
-                        if (t > 0) dk::mbar_wait(&rec_empty[which], (t - 1) & 1);
+                        if (t > 0) twait(&rec_empty[which], (t - 1) & 1, tr, tw1);
                         issue_box(which, nx++);
                     }
                 };
@@ -316,7 +360,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
             for (int ti = 0; ti < n_tiles; ti++) {
                 const int tile = tile_begin + ti;
                 const int rs = ti % a.n_rec_stages, ruse = ti / a.n_rec_stages;
-                if (ruse > 0) dk::mbar_wait(&rec_empty[rs], (ruse - 1) & 1);
+                if (ruse > 0) twait(&rec_empty[rs], (ruse - 1) & 1, tr, tw1);
                 const int tx = tile % a.ntx, ty = (tile / a.ntx) % a.nty, tz = tile / (a.ntx * a.nty);
                 unsigned char* rdst = rec_smem + static_cast<size_t>(rs) * a.rec_stage_bytes;
                 if (elect_one()) {
@@ -327,7 +371,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                 }
                 __syncwarp();
                 for (int s = 0; s < a.nsteps; s += KS) {
-                    if (wuse >= a.wstages) dk::mbar_wait(&w_empty[ws], wph ^ 1);
+                    if (wuse >= a.wstages) twait(&w_empty[ws], wph ^ 1, tr, tw0);
                     if (elect_one()) {
                         dk::mbar_arrive_expect_tx(&w_full[ws], STAGE);
                         if constexpr (CL == 1) {
@@ -349,6 +393,14 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                 }
             }
             }   // !PAIR
+            if (tr && elect_one()) {
+                atomicAdd(&a.trace[TR_PROD_TOTAL], static_cast<unsigned long long>(clock64() - tstart));
+                atomicAdd(&a.trace[TR_PROD_WEMPTY], static_cast<unsigned long long>(tw0));
+                atomicAdd(&a.trace[TR_PROD_REMPTY], static_cast<unsigned long long>(tw1));
+                atomicAdd(&a.trace[TR_CTAS], 1ull);
+                atomicAdd(&a.trace[TR_TILES], static_cast<unsigned long long>(n_tiles));
+            }
+            __syncwarp();
             if constexpr (CL > 1) {
                 // drain: every ring slot's last release (from both MMA warps) has arrived before exit
                 for (int i = 0; i < min(wuse, a.wstages); i++) {
@@ -371,6 +423,86 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
             const uint64_t dP0 = umma_desc(rec0 + (PAIR ? a.rec_stage_bytes : 0), 32, 128);
             const uint32_t row16 = static_cast<uint32_t>(a.TXB) * 16u;
             const uint32_t rowTY = static_cast<uint32_t>(a.TYB) * row16;
+            if constexpr (PAIR && CL == 1) {
+            // Lean issue loop: one thread runs the whole schedule (no per-stage warp re-convergence), the
+            // stage loops are unrolled so every descriptor offset is an immediate; the tcgen05 queue stays fed.
+            constexpr int S1 = M * M * MXP, S1P = (S1 + KS - 1) / KS * KS;
+            constexpr int S2 = M * M * MXQ, S2P = (S2 + KS - 1) / KS * KS;
+            constexpr uint32_t ROW16 = static_cast<uint32_t>(pair_txb(M)) * 16u;
+            constexpr uint32_t ROWTY = static_cast<uint32_t>(Q + M - 1) * ROW16;
+            if (elect_one()) {
+                uint32_t ws = 0, wph = 0;
+                const uint32_t nws = static_cast<uint32_t>(a.wstages);
+                for (int ti = 0; ti < n_tiles; ti++) {
+                    const int buf = ti % NBUF, buse = ti / NBUF;
+                    const uint32_t dcol = tmem + static_cast<uint32_t>(buf * Q * NT);
+                    twait(&rec_full[0], ti & 1, tr, tw2);
+                    tc_fence_after();
+#pragma unroll
+                    for (int st = 0; st < S1P / KS; st++) {
+                        twait(&w_full[ws], wph, tr, tw1);
+                        tc_fence_after();
+                        const uint64_t da0 = dA0 + ((ws * STAGE) >> 4);
+                        if (st == 0 && buse > 0) {
+                            // accumulator rows are released one by one while the epilogue drains them
+#pragma unroll
+                            for (int q = 0; q < Q; q++) {
+                                twait(&tm_empty[buf * Q + q], (buse - 1) & 1, tr, tw0);
+                                tc_fence_after();
+#pragma unroll
+                                for (int ks = 0; ks < KS; ks++)
+                                    umma_bf16(dcol + q * NT, da0 + ((ks * WCHUNK) >> 4),
+                                              dB0 + ((pair_off1(M, ks, ROW16, ROWTY) + q * ROW16) >> 4), idesc,
+                                              ks == 0 ? 0u : 1u);
+                            }
+                        } else {
+#pragma unroll
+                            for (int ks = 0; ks < KS; ks++)
+#pragma unroll
+                                for (int q = 0; q < Q; q++)
+                                    umma_bf16(dcol + q * NT, da0 + ((ks * WCHUNK) >> 4),
+                                              dB0 + ((pair_off1(M, st * KS + ks, ROW16, ROWTY) + q * ROW16) >> 4),
+                                              idesc, (st == 0 && ks == 0) ? 0u : 1u);
+                        }
+                        umma_commit(&w_empty[ws]);
+                        if (++ws == nws) {
+                            ws = 0;
+                            wph ^= 1;
+                        }
+                    }
+                    umma_commit(&rec_empty[0]);
+                    twait(&rec_full[1], ti & 1, tr, tw2);
+                    tc_fence_after();
+#pragma unroll
+                    for (int st = 0; st < S2P / KS; st++) {
+                        twait(&w_full[ws], wph, tr, tw1);
+                        tc_fence_after();
+                        const uint64_t da0 = dA0 + ((ws * STAGE) >> 4);
+#pragma unroll
+                        for (int ks = 0; ks < KS; ks++)
+#pragma unroll
+                            for (int q = 0; q < Q; q++)
+                                umma_bf16(dcol + q * NT, da0 + ((ks * WCHUNK) >> 4),
+                                          dP0 + ((pair_off2(M, st * KS + ks, ROW16, ROWTY) + q * ROW16) >> 4), idesc,
+                                          1u);
+                        umma_commit(&w_empty[ws]);
+                        if (++ws == nws) {
+                            ws = 0;
+                            wph ^= 1;
+                        }
+                    }
+                    umma_commit(&rec_empty[1]);
+                    umma_commit(&tm_full[buf]);
+                }
+                if (tr) {
+                    atomicAdd(&a.trace[TR_MMA_TOTAL], static_cast<unsigned long long>(clock64() - tstart));
+                    atomicAdd(&a.trace[TR_MMA_TMEMPTY], static_cast<unsigned long long>(tw0));
+                    atomicAdd(&a.trace[TR_MMA_WFULL], static_cast<unsigned long long>(tw1));
+                    atomicAdd(&a.trace[TR_MMA_RFULL], static_cast<unsigned long long>(tw2));
+                }
+            }
+            __syncwarp();
+            } else {
             int ws = 0, wph = 0;
             // B descriptor of K-step s: PAIR pass 1 (kind 0), PAIR pass 2 (kind 1) or the 2-pass scheme (kind 2)
             auto bdesc = [&](int kind, int s, uint32_t rofs) -> uint64_t {
@@ -388,11 +520,27 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                 const int g = s / (MXP * M * M * 2);
                 return dB0 + ((rofs + g * a.box_bytes + vz * rowTY + vy * row16 + vxp * 32u) >> 4);
             };
-            auto issue_stage = [&](int kind, int s0, uint32_t rofs, uint32_t dcol, bool first) {
-                dk::mbar_wait(&w_full[ws], wph);
+            // rel != nullptr: first stage of a tile whose accumulator rows are still being drained --
+            // issue row-major, each row right after the epilogue released it (rel[q], parity relph)
+            auto issue_stage = [&](int kind, int s0, uint32_t rofs, uint32_t dcol, bool first, uint64_t* rel,
+                                   int relph) {
+                twait(&w_full[ws], wph, tr, tw1);
                 tc_fence_after();
-                if (elect_one()) {
-                    const uint64_t da0 = dA0 + ((static_cast<uint32_t>(ws) * STAGE) >> 4);
+                const uint64_t da0 = dA0 + ((static_cast<uint32_t>(ws) * STAGE) >> 4);
+                if (rel) {
+#pragma unroll
+                    for (int q = 0; q < Q; q++) {
+                        twait(&rel[q], relph, tr, tw0);
+                        tc_fence_after();
+                        if (elect_one()) {
+#pragma unroll
+                            for (int ks = 0; ks < KS; ks++)
+                                umma_bf16(dcol + q * NT, da0 + ((ks * WCHUNK) >> 4),
+                                          bdesc(kind, s0 + ks, rofs) + ((q * row16) >> 4), idesc, ks == 0 ? 0u : 1u);
+                        }
+                        __syncwarp();
+                    }
+                } else if (elect_one()) {
 #pragma unroll
                     for (int ks = 0; ks < KS; ks++) {
                         const uint64_t db = bdesc(kind, s0 + ks, rofs);
@@ -401,6 +549,9 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                         for (int q = 0; q < Q; q++)
                             umma_bf16(dcol + q * NT, da, db + ((q * row16) >> 4), idesc, (first && ks == 0) ? 0u : 1u);
                     }
+                }
+                __syncwarp();
+                if (elect_one()) {
                     if constexpr (CL == 1) umma_commit(&w_empty[ws]);
                     else umma_commit_mc(&w_empty[ws], CMASK);
                 }
@@ -414,15 +565,16 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                 const int buf = ti % NBUF, buse = ti / NBUF;
                 const uint32_t dcol = tmem + static_cast<uint32_t>(buf * Q * NT);
                 if constexpr (PAIR) {
-                    dk::mbar_wait(&rec_full[0], ti & 1);
-                    if (buse > 0) dk::mbar_wait(&tm_empty[buf], (buse - 1) & 1);
+                    twait(&rec_full[0], ti & 1, tr, tw2);
                     tc_fence_after();
-                    for (int s = 0; s < a.S1p; s += KS) issue_stage(0, s, 0u, dcol, s == 0);
+                    uint64_t* rel = buse > 0 ? &tm_empty[buf * Q] : nullptr;
+                    for (int s = 0; s < a.S1p; s += KS)
+                        issue_stage(0, s, 0u, dcol, s == 0, s == 0 ? rel : nullptr, (buse - 1) & 1);
                     if (elect_one()) umma_commit(&rec_empty[0]);
                     __syncwarp();
-                    dk::mbar_wait(&rec_full[1], ti & 1);
+                    twait(&rec_full[1], ti & 1, tr, tw2);
                     tc_fence_after();
-                    for (int s = 0; s < a.S2p; s += KS) issue_stage(1, s, 0u, dcol, false);
+                    for (int s = 0; s < a.S2p; s += KS) issue_stage(1, s, 0u, dcol, false, nullptr, 0);
                     if (elect_one()) {
                         umma_commit(&rec_empty[1]);
                         umma_commit(&tm_full[buf]);
@@ -430,11 +582,12 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                     __syncwarp();
                 } else {
                     const int rs = ti % a.n_rec_stages, ruse = ti / a.n_rec_stages;
-                    dk::mbar_wait(&rec_full[rs], ruse & 1);
-                    if (buse > 0) dk::mbar_wait(&tm_empty[buf], (buse - 1) & 1);
+                    twait(&rec_full[rs], ruse & 1, tr, tw2);
                     tc_fence_after();
                     const uint32_t rofs = static_cast<uint32_t>(rs * a.rec_stage_bytes);
-                    for (int s = 0; s < a.nsteps; s += KS) issue_stage(2, s, rofs, dcol, s == 0);
+                    uint64_t* rel = buse > 0 ? &tm_empty[buf * Q] : nullptr;
+                    for (int s = 0; s < a.nsteps; s += KS)
+                        issue_stage(2, s, rofs, dcol, s == 0, s == 0 ? rel : nullptr, (buse - 1) & 1);
                     if (elect_one()) {
                         umma_commit(&tm_full[buf]);
                         umma_commit(&rec_empty[rs]);
@@ -442,11 +595,25 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                     __syncwarp();
                 }
             }
+            if (tr && elect_one()) {
+                atomicAdd(&a.trace[TR_MMA_TOTAL], static_cast<unsigned long long>(clock64() - tstart));
+                atomicAdd(&a.trace[TR_MMA_TMEMPTY], static_cast<unsigned long long>(tw0));
+                atomicAdd(&a.trace[TR_MMA_WFULL], static_cast<unsigned long long>(tw1));
+                atomicAdd(&a.trace[TR_MMA_RFULL], static_cast<unsigned long long>(tw2));
+            }
+            __syncwarp();
+            }   // generic issue loop
         } else {
             // ------------------------------------------------ epilogue warps
+            // Warp (quarter, class cls) reads TMEM lanes of its quarter (lane = rotation).  Rows are
+            // drained in order q = 0..Q-1 so each accumulator row is released (tm_empty[buf][q]) as soon as
+            // its last chunk is in registers, before the chunk is processed; within row q the warp takes the
+            // 32-column chunks c = (q + cls + j * nclass) mod 4 ("diagonal" classes: over the Q rows of a
+            // tile a class covers one chunk per row, so the cells of a list are spread like a row class).
             const int quarter = warp & 3;
-            const int half = (warp - 2) >> 2;         // row class of this warp
+            const int cls = (warp - 2) >> 2;
             const int nclass = a.nepi >> 2;
+            constexpr int NCH = NT / 32;                         // 32-column chunks per row
             const int r = quarter * 32 + lane;                  // rotation within the block (TMEM lane)
             const int slot = block * ROT + r;
             const bool rot_ok = slot < a.n_slots;
@@ -455,50 +622,63 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
             for (int i = 0; i < LIST; i++) lst[i] = KEY_MAX;
             float th = __int_as_float(0x7f800000);   // score of the list's last key (+inf while not full)
             uint32_t th_t = 0xffffffffu;             // t_lin of the list's last key
+            int tx = tile_begin % a.ntx, ty = (tile_begin / a.ntx) % a.nty, tz = tile_begin / (a.ntx * a.nty);
             for (int ti = 0; ti < n_tiles; ti++) {
-                const int tile = tile_begin + ti;
                 const int buf = ti % NBUF, buse = ti / NBUF;
-                dk::mbar_wait(&tm_full[buf], buse & 1);
+                twait(&tm_full[buf], buse & 1, tr, tw0);
                 tc_fence_after();
-                const int tx = tile % a.ntx, ty = (tile / a.ntx) % a.nty, tz = tile / (a.ntx * a.nty);
-                for (int q = half; q < Q; q += nclass) {
-                    const int y = ty * Q + q, z = tz;
-                    const bool row_ok = rot_ok && y < a.ny && z < a.nz;
+                if (a.dbg == 1) {   // diagnostic: no TMEM drain
+                    __syncwarp();
+                    if (lane == 0)
+                        for (int q = 0; q < Q; q++) dk::mbar_arrive(&tm_empty[buf * Q + q]);
+                } else {
                     const int x0 = tx * NT;
-                    const uint32_t tbase = static_cast<uint32_t>((z * a.ny + y) * a.nx + x0);
+                    for (int q = 0; q < Q; q++) {
+                        const int y = ty * Q + q, z = tz;
+                        const bool row_ok = rot_ok && y < a.ny && z < a.nz;
+                        const uint32_t tbase = static_cast<uint32_t>((z * a.ny + y) * a.nx + x0);
 #pragma unroll 1
-                    for (int c0 = 0; c0 < NT; c0 += 32) {
-                        uint32_t v[32];
-                        tmem_ld32(tmem + (static_cast<uint32_t>(quarter * 32) << 16) + (buf * Q + q) * NT + c0, v);
-                        if (!row_ok) continue;
-                        if constexpr (GRID) {
-                            float* out = a.grid + static_cast<size_t>(slot) * a.nx * a.ny * a.nz + tbase;
+                        for (int j = 0; j < NCH / nclass; j++) {
+                            const int c0 = ((q + cls + j * nclass) & (NCH - 1)) * 32;
+                            uint32_t v[32];
+                            const long long tl0 = tr ? clock64() : 0;
+                            tmem_ld32(tmem + (static_cast<uint32_t>(quarter * 32) << 16) + (buf * Q + q) * NT + c0, v);
+                            if (tr) tw1 += clock64() - tl0;
+                            if (j == NCH / nclass - 1) {   // the row's last chunk is in registers: release the row
+                                tc_fence_before();
+                                __syncwarp();
+                                if (lane == 0) dk::mbar_arrive(&tm_empty[buf * Q + q]);
+                            }
+                            if (!row_ok || a.dbg == 2) continue;
+                            if constexpr (GRID) {
+                                float* out = a.grid + static_cast<size_t>(slot) * a.nx * a.ny * a.nz + tbase;
 #pragma unroll
-                            for (int j = 0; j < 32; j++)
-                                if (x0 + c0 + j < a.nx) out[c0 + j] = __uint_as_float(v[j]);
-                        } else {
-                            // fast check: one FMNMX per value; the insertion path is rare after warm-up
-                            float mn = __uint_as_float(v[0]);
+                                for (int jj = 0; jj < 32; jj++)
+                                    if (x0 + c0 + jj < a.nx) out[c0 + jj] = __uint_as_float(v[jj]);
+                            } else {
+                                // fast check: one FMNMX per value; the insertion path is rare after warm-up
+                                float mn = __uint_as_float(v[0]);
 #pragma unroll
-                            for (int j = 1; j < 32; j++) mn = fminf(mn, __uint_as_float(v[j]));
-                            // exact gate: a strictly better score, or a tie that could carry a smaller t_lin
-                            if (mn < th || (mn == th && tbase + c0 < th_t)) {
-                                // rare path: bitmask of candidates, each extracted with a 5-level select tree
-                                const int jmax = min(32, a.nx - x0 - c0);
-                                uint32_t msk = 0;
+                                for (int jj = 1; jj < 32; jj++) mn = fminf(mn, __uint_as_float(v[jj]));
+                                // exact gate: a strictly better score, or a tie that could carry a smaller t_lin
+                                if (mn < th || (mn == th && tbase + c0 < th_t)) {
+                                    // rare path: bitmask of candidates, each extracted with a 5-level select tree
+                                    const int jmax = min(32, a.nx - x0 - c0);
+                                    uint32_t msk = 0;
 #pragma unroll
-                                for (int j = 0; j < 32; j++)
-                                    msk |= (__uint_as_float(v[j]) <= th && j < jmax) ? (1u << j) : 0u;
-                                while (msk) {
-                                    const int j = __ffs(msk) - 1;
-                                    msk &= msk - 1;
-                                    const float sv = __uint_as_float(select32(v, j));
-                                    if (sv <= th) {
-                                        const unsigned long long key = dk::make_key(sv, tbase + c0 + j);
-                                        if (key < lst[LIST - 1]) {
-                                            list_insert(lst, key);
-                                            th = dk::key_score_bound(static_cast<uint32_t>(lst[LIST - 1] >> 32));
-                                            th_t = static_cast<uint32_t>(lst[LIST - 1] & 0xffffffffu);
+                                    for (int jj = 0; jj < 32; jj++)
+                                        msk |= (__uint_as_float(v[jj]) <= th && jj < jmax) ? (1u << jj) : 0u;
+                                    while (msk) {
+                                        const int jj = __ffs(msk) - 1;
+                                        msk &= msk - 1;
+                                        const float sv = __uint_as_float(select32(v, jj));
+                                        if (sv <= th) {
+                                            const unsigned long long key = dk::make_key(sv, tbase + c0 + jj);
+                                            if (key < lst[LIST - 1]) {
+                                                list_insert(lst, key);
+                                                th = dk::key_score_bound(static_cast<uint32_t>(lst[LIST - 1] >> 32));
+                                                th_t = static_cast<uint32_t>(lst[LIST - 1] & 0xffffffffu);
+                                            }
                                         }
                                     }
                                 }
@@ -506,9 +686,19 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                         }
                     }
                 }
-                tc_fence_before();
-                __syncwarp();
-                if (lane == 0) dk::mbar_arrive(&tm_empty[buf]);
+                if (++tx == a.ntx) {
+                    tx = 0;
+                    if (++ty == a.nty) {
+                        ty = 0;
+                        tz++;
+                    }
+                }
+            }
+            if (tr && lane == 0) {
+                atomicAdd(&a.trace[TR_EPI_TOTAL], static_cast<unsigned long long>(clock64() - tstart));
+                atomicAdd(&a.trace[TR_EPI_TMFULL], static_cast<unsigned long long>(tw0));
+                atomicAdd(&a.trace[TR_EPI_LDTM], static_cast<unsigned long long>(tw1));
+                atomicAdd(&a.trace[TR_EPI_WARPS], 1ull);
             }
             if constexpr (!GRID) {
                 if (rot_ok) {
@@ -808,6 +998,8 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc2(const __grid_constant_
     cluster_sync_all();
     tc_fence_after();
     const uint32_t tmem = tmem_base_s;
+    const bool tr = a.trace != nullptr;
+    long long tw0 = 0, tw1 = 0, tw2 = 0, tstart = tr ? clock64() : 0;
 
     if (n_tiles > 0) {
         if (warp == 0) {
@@ -820,7 +1012,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc2(const __grid_constant_
             int ws = 0, wph = 0, wuse = 0;
             auto stream_weights = [&](int s0, int s1) {
                 for (int s = s0; s < s1; s += KS) {
-                    if (wuse >= a.wstages) dk::mbar_wait(&w_empty[ws], wph ^ 1);
+                    if (wuse >= a.wstages) twait(&w_empty[ws], wph ^ 1, tr, tw0);
                     if (elect_one()) {
                         dk::mbar_arrive_expect_tx(&w_full[ws], STAGE);
                         dk::bulk_load(w_smem + static_cast<size_t>(ws) * STAGE, wsrc + static_cast<size_t>(s) * WCHUNK,
@@ -855,7 +1047,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc2(const __grid_constant_
             auto ensure = [&](int which, int t) {
                 int& nx = which ? pp : pm;
                 if (nx == t) {
-                    if (t > 0) dk::mbar_wait(&rec_empty[which], (t - 1) & 1);
+                    if (t > 0) twait(&rec_empty[which], (t - 1) & 1, tr, tw1);
                     issue_box(which, nx++);
                 }
             };
@@ -871,6 +1063,14 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc2(const __grid_constant_
                     stream_weights(s, s + KS);
                 }
             }
+            if (tr && leader && elect_one()) {
+                atomicAdd(&a.trace[TR_PROD_TOTAL], static_cast<unsigned long long>(clock64() - tstart));
+                atomicAdd(&a.trace[TR_PROD_WEMPTY], static_cast<unsigned long long>(tw0));
+                atomicAdd(&a.trace[TR_PROD_REMPTY], static_cast<unsigned long long>(tw1));
+                atomicAdd(&a.trace[TR_CTAS], 1ull);
+                atomicAdd(&a.trace[TR_TILES], static_cast<unsigned long long>(n_tiles));
+            }
+            __syncwarp();
         } else if (warp == 1) {
             if (!leader) {
                 // ------------------------------------------------ relay: tell the leader our stages landed
@@ -908,8 +1108,8 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc2(const __grid_constant_
                 const uint32_t rowTY = static_cast<uint32_t>(a.TYB) * row16;
                 int ws = 0, wph = 0;
                 auto issue_stage = [&](int kind, int s0, bool first) {
-                    dk::mbar_wait(&w_full[ws], wph);
-                    dk::mbar_wait(&peer_w[ws], wph);
+                    twait(&w_full[ws], wph, tr, tw1);
+                    twait(&peer_w[ws], wph, tr, tw1);
                     tc_fence_after();
                     if (elect_one()) {
                         const uint64_t da0 = dA0 + ((static_cast<uint32_t>(ws) * STAGE) >> 4);
@@ -939,15 +1139,15 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc2(const __grid_constant_
                     }
                 };
                 for (int ti = 0; ti < n_tiles; ti++) {
-                    dk::mbar_wait(&rec_full[0], ti & 1);
-                    dk::mbar_wait(&peer_rec[0], ti & 1);
-                    if (ti > 0) dk::mbar_wait(&tm_empty[0], (ti - 1) & 1);
+                    twait(&rec_full[0], ti & 1, tr, tw2);
+                    twait(&peer_rec[0], ti & 1, tr, tw2);
+                    if (ti > 0) twait(&tm_empty[0], (ti - 1) & 1, tr, tw0);
                     tc_fence_after();
                     for (int s = 0; s < a.S1p; s += KS) issue_stage(0, s, s == 0);
                     if (elect_one()) umma_commit_2sm_mc(&rec_empty[0], PAIRMASK);
                     __syncwarp();
-                    dk::mbar_wait(&rec_full[1], ti & 1);
-                    dk::mbar_wait(&peer_rec[1], ti & 1);
+                    twait(&rec_full[1], ti & 1, tr, tw2);
+                    twait(&peer_rec[1], ti & 1, tr, tw2);
                     tc_fence_after();
                     for (int s = 0; s < a.S2p; s += KS) issue_stage(1, s, false);
                     if (elect_one()) {
@@ -956,6 +1156,13 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc2(const __grid_constant_
                     }
                     __syncwarp();
                 }
+                if (tr && elect_one()) {
+                    atomicAdd(&a.trace[TR_MMA_TOTAL], static_cast<unsigned long long>(clock64() - tstart));
+                    atomicAdd(&a.trace[TR_MMA_TMEMPTY], static_cast<unsigned long long>(tw0));
+                    atomicAdd(&a.trace[TR_MMA_WFULL], static_cast<unsigned long long>(tw1));
+                    atomicAdd(&a.trace[TR_MMA_RFULL], static_cast<unsigned long long>(tw2));
+                }
+                __syncwarp();
             }
         } else if (warp < 2 + a.nepi) {
             // ------------------------------------------------ epilogue warps (both CTAs)
@@ -972,8 +1179,16 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc2(const __grid_constant_
             uint32_t th_t = 0xffffffffu;
             for (int ti = 0; ti < n_tiles; ti++) {
                 const int tile = tile_begin + ti;
-                dk::mbar_wait(&tm_full[0], ti & 1);
+                twait(&tm_full[0], ti & 1, tr, tw0);
                 tc_fence_after();
+                if (a.dbg == 1) {   // diagnostic: no TMEM drain
+                    __syncwarp();
+                    if (lane == 0) {
+                        if (leader) dk::mbar_arrive(&tm_empty[0]);
+                        else mbar_arrive_remote(&tm_empty[0], 0);
+                    }
+                    continue;
+                }
                 const int tx = tile % a.ntx, ty = (tile / a.ntx) % a.nty, tz = tile / (a.ntx * a.nty);
                 for (int c4 = cls; c4 < 4; c4 += nclass) {
                     const int q = c4 >> 1, half = c4 & 1;
@@ -984,8 +1199,10 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc2(const __grid_constant_
 #pragma unroll 1
                     for (int c0 = 0; c0 < NT; c0 += 32) {
                         uint32_t v[32];
+                        const long long tl0 = tr ? clock64() : 0;
                         tmem_ld32(tmem + (static_cast<uint32_t>(quarter * 32) << 16) + q * 2 * NT + half * NT + c0, v);
-                        if (!row_ok) continue;
+                        if (tr) tw1 += clock64() - tl0;
+                        if (!row_ok || a.dbg == 2) continue;
                         if constexpr (GRID) {
                             float* out = a.grid + static_cast<size_t>(slot) * a.nx * a.ny * a.nz + tbase;
 #pragma unroll
@@ -1024,6 +1241,12 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc2(const __grid_constant_
                     if (leader) dk::mbar_arrive(&tm_empty[0]);
                     else mbar_arrive_remote(&tm_empty[0], 0);
                 }
+            }
+            if (tr && leader && lane == 0) {
+                atomicAdd(&a.trace[TR_EPI_TOTAL], static_cast<unsigned long long>(clock64() - tstart));
+                atomicAdd(&a.trace[TR_EPI_TMFULL], static_cast<unsigned long long>(tw0));
+                atomicAdd(&a.trace[TR_EPI_LDTM], static_cast<unsigned long long>(tw1));
+                atomicAdd(&a.trace[TR_EPI_WARPS], 1ull);
             }
             if constexpr (!GRID) {
                 if (rot_ok) {
