@@ -52,7 +52,7 @@ def parse():
                     help="correlation engine: auto (tcgen05 when eligible), ffma (FP32 FFMA), tc (tcgen05 bf16x3)")
     ap.add_argument("--no-alt", action="store_true", help="skip the secondary measurement of the other engine")
     ap.add_argument("--tc-epi", type=int, default=0, choices=[0, 4, 8, 16], help="tcgen05 epilogue warps (0 auto)")
-    ap.add_argument("--tc-variant", type=int, default=0, choices=[0, 1, 2, 3, 4],
+    ap.add_argument("--tc-variant", type=int, default=0, choices=[0, 1, 2, 3, 4, 5, 6],
                     help="tcgen05 tiling: 0 auto, 1 = 4 rows x 1 TMEM buffer, 2 = CTA pair, 2 rows x 2 buffers")
     return ap.parse_args()
 

@@ -138,7 +138,9 @@ typedef enum {
     DOCK_TUNE_ENGINE = 4,         /* correlation engine: 0 auto (tcgen05 when eligible), 1 FP32 FFMA, 2 tcgen05 */
     DOCK_TUNE_TC_VARIANT = 5,     /* tcgen05 tiling: 0 auto, 1 = 4 rows x 1 TMEM buffer, 2 = 2 rows x 2 buffers on a
                                      CTA pair with multicast weight streaming, 3 = cta_group::2 (M = 256 rotations,
-                                     N = 256 translations over a CTA pair), 4 = 2 rows x 2 TMEM buffers, single CTA */
+                                     N = 256 translations over a CTA pair), 4 = 2 rows x 2 TMEM buffers, single CTA,
+                                     5 / 6 = row-skewed schedule (rows one weight stage apart, drained while the
+                                     other rows compute) with 4 rows x 1 / 2 rows x 2 TMEM buffers */
     DOCK_TUNE_TC_EPILOGUE_WARPS = 6 /* tcgen05 epilogue warps: 0 auto (one translation row per thread), 4, 8, 16 */
 } dock_tune_key;
 
@@ -159,7 +161,7 @@ typedef struct {
     int n_sms;                 /* multiprocessors of the context's device */
     int engine_last;           /* engine of the last correlation: 1 FP32 FFMA, 2 tcgen05 bf16x3 */
     int tc_available;          /* 1 if the tcgen05 engine is available for m_max */
-    int tc_variant_last;       /* tcgen05 variant of the last correlation (1 or 2), 0 if FFMA */
+    int tc_variant_last;       /* tcgen05 variant of the last correlation (1..6), 0 if FFMA */
     int tc_ksteps_last;        /* K-steps (K = 16 each) per translation row executed by the last tcgen05 launch */
 } dock_info;
 

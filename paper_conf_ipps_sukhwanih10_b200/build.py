@@ -1,6 +1,7 @@
 """Build libdock.so in-tree with nvcc for sm_100a (no JIT, no torch extension cache)."""
 from __future__ import annotations
 
+import glob
 import os
 import subprocess
 import sys
@@ -10,7 +11,7 @@ ROOT = os.path.dirname(PKG)
 CSRC = os.path.join(PKG, "csrc")
 LIB = os.path.join(PKG, "libdock.so")
 SOURCES = [os.path.join(CSRC, "dock.cu")]
-HEADERS = [os.path.join(CSRC, "dock_kernels.cuh"), os.path.join(CSRC, "dock_tc.cuh"), os.path.join(ROOT, "include", "dock.h")]
+HEADERS = sorted(glob.glob(os.path.join(CSRC, "*.cuh"))) + [os.path.join(ROOT, "include", "dock.h")]
 
 NVCC_FLAGS = [
     "-gencode", "arch=compute_100a,code=sm_100a",

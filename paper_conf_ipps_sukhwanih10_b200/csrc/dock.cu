@@ -20,6 +20,7 @@
 #include "dock.h"
 #include "dock_kernels.cuh"
 #include "dock_tc.cuh"
+#include "dock_tc_skew.cuh"
 
 static_assert(sizeof(dock_pose) == 16, "dock_pose must be 16 bytes");
 static_assert(sizeof(dk::PoseOut) == sizeof(dock_pose), "kernel pose layout mismatch");
@@ -75,7 +76,7 @@ struct dock_ctx {
     uint16_t* d_rec_tc = nullptr;
     uint16_t* d_rec_pair = nullptr;   // PAIR-scheme receptor copy (P <= 4)
     int tc_Gch = 0, tc_ntx = 0, tc_ntz = 0, tc_Xp = 0, tc_Yp = 0, tc_Zp = 0;
-    TcPlan tcplan[5][DOCK_MAX_M + 1];   // [variant][m]
+    TcPlan tcplan[7][DOCK_MAX_M + 1];   // [variant][m]
     DevBuf Wtc;
     // diagnostics (environment, read at init): DOCK_TC_TRACE=1 prints per-role cycle counters of every
     // k_corr_tc launch to stderr; DOCK_TC_DEBUG=1|2 disables parts of the epilogue (timing only)
@@ -278,12 +279,15 @@ cudaError_t launch_corr(int m, const MPlan& pl, const dk::CorrArgs& a, int grid,
 }
 
 int tc_txb(int m) { return tc::NT + (m + 1) / 2 * 2 - 1; }
-// tcgen05 variants: 1 = Q4 rows x 1 TMEM buffer, single CTA; 2 = Q2 rows x 2 buffers, CTA pair + multicast.
-// tile rows (translation rows per tile): variants 1 and 3 tile 4 rows, variants 2 and 4 tile 2
-inline int tc_q(int v) { return (v == 2 || v == 4) ? 2 : 4; }
-inline int tc_cl(int v) { return (v == 1 || v == 4) ? 1 : 2; }
+// tcgen05 variants: 1 = Q4 rows x 1 TMEM buffer, single CTA; 2 = Q2 rows x 2 buffers, CTA pair + multicast;
+// 3 = cta_group::2 (4 rows over a CTA pair); 4 = Q2 x 2 buffers, single CTA; 5 / 6 = the row-skewed schedule
+// (dock_tc_skew.cuh) with Q4 x 1 buffer / Q2 x 2 buffers and z-plane receptor staging.
+// tile rows (translation rows per tile): variants 1, 3 and 5 tile 4 rows, the others 2
+inline int tc_q(int v) { return (v == 2 || v == 4 || v == 6) ? 2 : 4; }
+inline int tc_cl(int v) { return (v == 2 || v == 3) ? 2 : 1; }
+inline bool tc_skew(int v) { return v == 5 || v == 6; }
 // receptor rows held per CTA (variant 3 splits the 4 tile rows over the CTA pair)
-inline int tc_rows_cta(int v) { return v == 1 ? 4 : 2; }
+inline int tc_rows_cta(int v) { return v == 3 ? 2 : tc_q(v); }
 inline int tc_nty(const dock_ctx* c, int v) { return (c->ny + tc_q(v) - 1) / tc_q(v); }
 inline int tc_ntiles(const dock_ctx* c, int v) { return c->tc_ntx * tc_nty(c, v) * c->tc_ntz; }
 
@@ -300,7 +304,8 @@ dock_status make_tc_plan(dock_ctx* ctx, int m, int v)
     // PAIR needs the (hi,lo) box and the (hi,hi') box resident together; otherwise the 2-pass scheme
     const int pair_box = round_up(16 * tc_txb_any(m) * (tc_rows_cta(v) + m - 1) * m, 1024);
     pl.pair = ctx->tc_Gch == 1 && ctx->d_rec_pair != nullptr && 2 * pair_box + min_ring <= budget;
-    if (!pl.pair && v != 1) return DOCK_OK;          // the CTA-pair variants are built for the PAIR scheme only
+    if (!pl.pair && v != 1) return DOCK_OK;          // variants 2-6 are built for the PAIR scheme only
+    if (tc_skew(v) && m < 3) return DOCK_OK;        // the skewed schedule needs >= Q weight stages per tile
     pl.TXB = pl.pair ? tc_txb_any(m) : tc_txb(m);
     pl.TYB = tc_rows_cta(v) + m - 1;
     pl.TZB = m;
@@ -309,6 +314,7 @@ dock_status make_tc_plan(dock_ctx* ctx, int m, int v)
     if (pl.pair && tc_cl(v) == 1 && (pl.TXB != tc::pair_txb(m) || pl.TYB != tc_q(v) + m - 1))
         return fail(ctx, DOCK_E_CUDA, "tcgen05 PAIR box geometry mismatch");
     pl.rec_stage_bytes = round_up(ctx->tc_Gch * pl.box_bytes, 1024);
+    if (tc_skew(v)) pl.rec_stage_bytes = round_up(m * (int)tc::plane_stride(m, tc_q(v)), 1024);
     if (pl.pair) {
         pl.S1 = m * m * ((m + 1) / 2);
         pl.S1p = round_up(pl.S1, KS);
@@ -323,6 +329,7 @@ dock_status make_tc_plan(dock_ctx* ctx, int m, int v)
     else if (!pl.pair && pl.rec_stage_bytes + min_ring <= budget) pl.n_rec_stages = 1;
     else return DOCK_OK;                    // this m is not eligible for the tensor-core engine
     pl.wstages = std::min(tc::WSTAGES, (budget - pl.n_rec_stages * pl.rec_stage_bytes) / stage);
+    if (tc_skew(v) && pl.wstages < tc_q(v) + 1) return DOCK_OK;   // every row holds one stage of the ring
     const int ring = pl.wstages * stage;
     // >= 116 KB keeps one CTA per SM: every CTA allocates all 512 TMEM columns
     pl.smem = std::max(pl.n_rec_stages * pl.rec_stage_bytes + ring, 116 * 1024);
@@ -331,7 +338,8 @@ dock_status make_tc_plan(dock_ctx* ctx, int m, int v)
     const cuuint64_t X = ctx->tc_Xp, Y = ctx->tc_Yp, Z = ctx->tc_Zp;
     cuuint64_t dims[5] = {8, X, Y, Z, (cuuint64_t)ctx->tc_Gch};
     cuuint64_t strides[4] = {16, X * 16, X * Y * 16, X * Y * Z * 16};
-    cuuint32_t box[5] = {8, (cuuint32_t)pl.TXB, (cuuint32_t)pl.TYB, (cuuint32_t)pl.TZB, 1};
+    // the skewed kernels stage the receptor one z-plane per TMA box
+    cuuint32_t box[5] = {8, (cuuint32_t)pl.TXB, (cuuint32_t)pl.TYB, (cuuint32_t)(tc_skew(v) ? 1 : pl.TZB), 1};
     cuuint32_t es[5] = {1, 1, 1, 1, 1};
     for (int which = 0; which < (pl.pair ? 2 : 1); which++) {
         CUresult r = fn(which ? &pl.tmap_pair : &pl.tmap, CU_TENSOR_MAP_DATA_TYPE_BFLOAT16, 5,
@@ -428,9 +436,35 @@ cudaError_t launch_tc2(int m, const TcPlan& pl, const tc::TcArgs& a, int grid, c
     }
 }
 
+template <int M, int Q, int NBUF, bool GRID>
+cudaError_t launch_skew_t(const TcPlan& pl, const tc::TcArgs& a, int grid, cudaStream_t st)
+{
+    auto kern = tc::k_corr_tc_skew<M, Q, NBUF, GRID>;
+    cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, pl.smem);
+    if (e != cudaSuccess) return e;
+    kern<<<grid, (2 + a.nepi) * 32, pl.smem, st>>>(pl.tmap, pl.tmap_pair, a);
+    return cudaGetLastError();
+}
+
+template <int Q, int NBUF, bool GRID>
+cudaError_t launch_skew(int m, const TcPlan& pl, const tc::TcArgs& a, int grid, cudaStream_t st)
+{
+    switch (m) {
+        case 3: return launch_skew_t<3, Q, NBUF, GRID>(pl, a, grid, st);
+        case 4: return launch_skew_t<4, Q, NBUF, GRID>(pl, a, grid, st);
+        case 5: return launch_skew_t<5, Q, NBUF, GRID>(pl, a, grid, st);
+        case 6: return launch_skew_t<6, Q, NBUF, GRID>(pl, a, grid, st);
+        case 7: return launch_skew_t<7, Q, NBUF, GRID>(pl, a, grid, st);
+        case 8: return launch_skew_t<8, Q, NBUF, GRID>(pl, a, grid, st);
+        default: return cudaErrorInvalidValue;
+    }
+}
+
 template <bool GRID>
 cudaError_t launch_tc(int m, int v, const TcPlan& pl, const tc::TcArgs& a, int grid, cudaStream_t st)
 {
+    if (v == 5) return launch_skew<4, 1, GRID>(m, pl, a, grid, st);
+    if (v == 6) return launch_skew<2, 2, GRID>(m, pl, a, grid, st);
     if (v == 3) return launch_tc2<GRID>(m, pl, a, grid, st);
     if (!pl.pair) return v == 1 ? launch_tc_v<1, false, GRID>(m, pl, a, grid, st) : cudaErrorInvalidValue;
     if (v == 4) return launch_tc_v<4, true, GRID>(m, pl, a, grid, st);
@@ -766,10 +800,12 @@ bool plan_tc_launch(dock_ctx* ctx, int m, int n_slots, int* v_out, int* G_out)
             return true;
         }
     }
-    if (ctx->tc_variant == 4 && ctx->tcplan[4][m].ok) {
-        *v_out = 4;
-        *G_out = choose_regions_n(ctx, n_blocks, tc_ntiles(ctx, 4));
-        return true;
+    for (int v : {4, 5, 6}) {
+        if (ctx->tc_variant == v && ctx->tcplan[v][m].ok) {
+            *v_out = v;
+            *G_out = choose_regions_n(ctx, n_blocks, tc_ntiles(ctx, v));
+            return true;
+        }
     }
     if (ctx->tc_variant == 3 && ctx->tcplan[3][m].ok) {
         // CTA pairs over pairs of rotation blocks; a pair occupies two SMs
@@ -1022,9 +1058,8 @@ dock_status dock_init(const dock_grid_desc* g, const float* receptor, const floa
     for (int m = 1; m <= ctx->m_max; m++) {
         dock_status s = make_plan(ctx, m);
         if (s != DOCK_OK && m == ctx->m_max) return bail(s);
-        if (make_tc_plan(ctx, m, 1) != DOCK_OK || make_tc_plan(ctx, m, 2) != DOCK_OK ||
-            make_tc_plan(ctx, m, 3) != DOCK_OK || make_tc_plan(ctx, m, 4) != DOCK_OK)
-            return bail(DOCK_E_CUDA);
+        for (int v = 1; v <= 6; v++)
+            if (make_tc_plan(ctx, m, v) != DOCK_OK) return bail(DOCK_E_CUDA);
     }
     *out = ctx;
     return DOCK_OK;
@@ -1044,7 +1079,7 @@ dock_status dock_set_tuning(dock_ctx* ctx, int key, int64_t value)
             ctx->engine = (int)value;
             return DOCK_OK;
         case DOCK_TUNE_TC_VARIANT:
-            if (value < 0 || value > 4) return fail(ctx, DOCK_E_INVALID_ARG, "tc variant must be 0..4");
+            if (value < 0 || value > 6) return fail(ctx, DOCK_E_INVALID_ARG, "tc variant must be 0..6");
             ctx->tc_variant = (int)value;
             return DOCK_OK;
         case DOCK_TUNE_TC_EPILOGUE_WARPS:

@@ -204,20 +204,19 @@ __host__ __device__ constexpr int pair_txb(int m)
                                                                      : (4 * ((m + 3) / 4) + 126);
 }
 // Byte offset of K-step s inside the PAIR pass-1 box ((hi,lo) voxels, 2 per K-step) and pass-2 box
-// ((hi(x),hi(x+1)) slots, 4 voxels per K-step); padding steps (zero weights) read the box origin.
+// ((hi(x),hi(x+1)) slots, 4 voxels per K-step); padding steps (zero weights) re-read the last real
+// step's voxels (a plane still resident in the z-plane pipeline of dock_tc_skew.cuh).
 __host__ __device__ constexpr uint32_t pair_off1(int m, int s, uint32_t row16, uint32_t rowTY)
 {
-    return s >= m * m * ((m + 1) / 2) ? 0u
-                                      : static_cast<uint32_t>(s / (((m + 1) / 2) * m)) * rowTY +
-                                            static_cast<uint32_t>((s / ((m + 1) / 2)) % m) * row16 +
-                                            static_cast<uint32_t>(s % ((m + 1) / 2)) * 32u;
+    const int mxp = (m + 1) / 2, t = s < m * m * mxp ? s : m * m * mxp - 1;
+    return static_cast<uint32_t>(t / (mxp * m)) * rowTY + static_cast<uint32_t>((t / mxp) % m) * row16 +
+           static_cast<uint32_t>(t % mxp) * 32u;
 }
 __host__ __device__ constexpr uint32_t pair_off2(int m, int s, uint32_t row16, uint32_t rowTY)
 {
-    return s >= m * m * ((m + 3) / 4) ? 0u
-                                      : static_cast<uint32_t>(s / (((m + 3) / 4) * m)) * rowTY +
-                                            static_cast<uint32_t>((s / ((m + 3) / 4)) % m) * row16 +
-                                            static_cast<uint32_t>(s % ((m + 3) / 4)) * 64u;
+    const int mxq = (m + 3) / 4, t = s < m * m * mxq ? s : m * m * mxq - 1;
+    return static_cast<uint32_t>(t / (mxq * m)) * rowTY + static_cast<uint32_t>((t / mxq) % m) * row16 +
+           static_cast<uint32_t>(t % mxq) * 64u;
 }
 
 // CL = 1: one CTA per item.  CL = 2: a cluster of two CTAs works on the same rotation block

@@ -29,8 +29,9 @@ def D():
 # engine ids used by the tests: 1 = FP32 FFMA; 2 = tcgen05 variant 1 (4 rows, 1 TMEM buffer);
 # 3 = tcgen05 variant 2 (2 rows, 2 TMEM buffers, CTA pair with multicast weights);
 # 4 = tcgen05 variant 3 (cta_group::2, M = 256 rotations x N = 256 translations over a CTA pair);
-# 5 = tcgen05 variant 4 (2 rows x 2 TMEM buffers, single CTA)
-ENGINES = [1, 2, 3, 4, 5]
+# 5 = tcgen05 variant 4 (2 rows x 2 TMEM buffers, single CTA);
+# 6, 7 = tcgen05 variants 5, 6 (row-skewed schedule, z-plane receptor staging; 4 rows x 1 / 2 rows x 2 buffers)
+ENGINES = [1, 2, 3, 4, 5, 6, 7]
 
 
 def _ctx(D, R, w, m_max, engine=0):
