@@ -16,6 +16,7 @@ reference arm of this tier) on bounded samples of the same workload.
 from __future__ import annotations
 
 import argparse
+import dataclasses
 import json
 import os
 import statistics
@@ -43,6 +44,8 @@ def parse():
     ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
     ap.add_argument("--config", default="prod", choices=sorted(g.CONFIGS))
     ap.add_argument("--k", type=int, default=None)
+    ap.add_argument("--rotations", type=int, default=0,
+                    help="override the config's rotation count (e.g. one rank's shard of the large config)")
     ap.add_argument("--rho", type=int, default=1)
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--no-cpu-baseline", action="store_true")
@@ -52,13 +55,15 @@ def parse():
                     help="correlation engine: auto (tcgen05 when eligible), ffma (FP32 FFMA), tc (tcgen05 bf16x3)")
     ap.add_argument("--no-alt", action="store_true", help="skip the secondary measurement of the other engine")
     ap.add_argument("--tc-epi", type=int, default=0, choices=[0, 4, 8, 16], help="tcgen05 epilogue warps (0 auto)")
-    ap.add_argument("--tc-variant", type=int, default=0, choices=[0, 1, 2, 3, 4, 5, 6],
-                    help="tcgen05 tiling: 0 auto, 1 = 4 rows x 1 TMEM buffer, 2 = CTA pair, 2 rows x 2 buffers")
+    ap.add_argument("--tc-variant", type=int, default=0, choices=[0, 1, 2],
+                    help="tcgen05 kernel: 0 auto, 1 = resident receptor boxes (P <= 4), 2 = streamed (group, z-plane) units")
     return ap.parse_args()
 
 
-def workload(cfg_name: str, k_override, rho: int):
+def workload(cfg_name: str, k_override, rho: int, n_rot_override: int = 0):
     c = g.CONFIGS[cfg_name]
+    if n_rot_override:
+        c = dataclasses.replace(c, n_rot=n_rot_override)
     k = k_override or c.k
     R = g.receptor_ftmap_like(c.n, c.P)
     w = g.weights(c.P)
@@ -159,7 +164,7 @@ def run_reference(args):
     rank = int(os.environ.get("RANK", "0"))
     if rank != 0:
         return
-    c, k, R, w, probes, rot, desc = workload(args.config, args.k, args.rho)
+    c, k, R, w, probes, rot, desc = workload(args.config, args.k, args.rho, args.rotations)
     n_units = c.n_probes * c.n_rot
     per_step = max(2.0, min(args.cpu_seconds, 120.0 / max(1, args.steps + args.warmup)))
     samples = []
@@ -197,16 +202,22 @@ def roofline(pk, pk_kind, info, c, flops_launch, corr_ms, ms_step, units_local):
     if info["engine_last"] == 2:
         peak = float(pk.get("bf16_tflops", 1590.0))
         ks = int(info.get("tc_ksteps_last", 0)) or 2 * c.m * c.m * ((c.m + 1) // 2)
-        # executed bf16 MMA FLOPs: K = 16 per step, ks steps per translation row (bf16x3 split + padding)
-        executed = flops_launch * (ks * 16.0) / (c.P * c.m ** 3)
+        # executed bf16 MMA FLOPs: K = 16 per step, ks steps per translation row (bf16x3 split + padding),
+        # times the x / y tiling waste of the launch's row width and rows per tile
+        ntt, q = int(info.get("tc_row_last", 128)) or 128, int(info.get("tc_rows_per_tile_last", 4)) or 4
+        nx, ny = c.n[0], c.n[1]
+        waste = (-(-nx // ntt) * ntt / nx) * (-(-ny // q) * q / ny)
+        executed = flops_launch * (ks * 16.0) / (c.P * c.m ** 3) * waste
         v = int(info.get("tc_variant_last", 1)) or 1
-        kname = {1: f"k_corr_tc<{c.m},4,1,1,PAIR,false>", 2: f"k_corr_tc<{c.m},2,2,2,PAIR,false>",
-                 3: f"k_corr_tc2<{c.m},false>", 4: f"k_corr_tc<{c.m},2,2,1,PAIR,false>"}.get(v, "k_corr_tc")
+        kname = f"k_corr_tc<{c.m},false>" if v == 1 else f"k_corr_tcs<{c.m},{ntt},{q},false>"
         return {"bound": "tensor", "engine": f"tcgen05 bf16x3 (variant {v})", "kernel": kname,
                 "achieved": achieved, "peak": peak, "unit": "TFLOP/s", "frac": achieved / peak, "traffic": None,
                 "peak_source": f"bf16 dense tensor peak, burst, MEASURED_PEAKS.json ({pk_kind})",
                 "executed_tensor_tflops": executed / (corr_ms / 1000.0) / 1e12,
                 "executed_frac": executed / (corr_ms / 1000.0) / 1e12 / peak,
+                # the measured cuBLAS figure was taken under the power cap; mostly-zero probe weights draw
+                # less power and keep this kernel at max SM clock, so it is also quoted against the nominal
+                "executed_frac_of_nominal_2250": executed / (corr_ms / 1000.0) / 1e12 / 2250.0,
                 "fp32_equiv_frac": achieved / (n_sms * 128 * 2 * float(pk.get("sm_max_mhz", 1965.0)) * 1e6 / 1e12),
                 "flops_per_launch": flops_launch, "launch_ms": corr_ms,
                 "kernel_share_of_step": corr_ms / ms_step if ms_step > 0 else None}
@@ -235,7 +246,7 @@ def run_ours(args):
         dist.init_process_group("nccl", device_id=torch.device("cuda", local))
     dev = torch.device("cuda", local)
 
-    c, k, R, w, probes, rot, desc = workload(args.config, args.k, args.rho)
+    c, k, R, w, probes, rot, desc = workload(args.config, args.k, args.rho, args.rotations)
     n_units = c.n_probes * c.n_rot
     b, e = parallel.shard_range(n_units, rank, world)
     ctx = D.dock_init(torch.from_numpy(R).to(dev), torch.from_numpy(w).to(dev), g.SPACING, m_max=c.m,

@@ -136,11 +136,11 @@ typedef enum {
     DOCK_TUNE_FORCE_FALLBACK = 2, /* 1 => every rotation takes the exact full-grid fallback (tests) */
     DOCK_TUNE_CAND_CAP = 3,       /* candidates kept per rotation before overflow fallback (>= 32) */
     DOCK_TUNE_ENGINE = 4,         /* correlation engine: 0 auto (tcgen05 when eligible), 1 FP32 FFMA, 2 tcgen05 */
-    DOCK_TUNE_TC_VARIANT = 5,     /* tcgen05 tiling: 0 auto, 1 = 4 rows x 1 TMEM buffer, 2 = 2 rows x 2 buffers on a
-                                     CTA pair with multicast weight streaming, 3 = cta_group::2 (M = 256 rotations,
-                                     N = 256 translations over a CTA pair), 4 = 2 rows x 2 TMEM buffers, single CTA,
-                                     5 / 6 = row-skewed schedule (rows one weight stage apart, drained while the
-                                     other rows compute) with 4 rows x 1 / 2 rows x 2 TMEM buffers */
+    DOCK_TUNE_TC_VARIANT = 5,     /* tcgen05 kernel: 0 auto, 1 = resident receptor boxes (one channel group, P <= 4,
+                                     128 translations x 4 rows per tile), 2 = receptor streamed one (channel group,
+                                     z-plane) unit at a time (any P <= 32, m <= 8; 64 / 128 / 160 translations per
+                                     row, chosen at init for nx).  A variant that cannot run m falls back to the
+                                     other one. */
     DOCK_TUNE_TC_EPILOGUE_WARPS = 6 /* tcgen05 epilogue warps: 0 auto (one translation row per thread), 4, 8, 16 */
 } dock_tune_key;
 
@@ -161,8 +161,10 @@ typedef struct {
     int n_sms;                 /* multiprocessors of the context's device */
     int engine_last;           /* engine of the last correlation: 1 FP32 FFMA, 2 tcgen05 bf16x3 */
     int tc_available;          /* 1 if the tcgen05 engine is available for m_max */
-    int tc_variant_last;       /* tcgen05 variant of the last correlation (1..6), 0 if FFMA */
+    int tc_variant_last;       /* tcgen05 variant of the last correlation (1 or 2), 0 if FFMA */
     int tc_ksteps_last;        /* K-steps (K = 16 each) per translation row executed by the last tcgen05 launch */
+    int tc_row_last;           /* translations per MMA row (MMA N) of the last tcgen05 launch */
+    int tc_rows_per_tile_last; /* translation rows per tile (TMEM accumulators) of the last tcgen05 launch */
 } dock_info;
 
 dock_status dock_get_info(const dock_ctx* ctx, dock_info* info);

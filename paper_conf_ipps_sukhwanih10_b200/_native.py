@@ -51,7 +51,8 @@ class dock_info(C.Structure):
                 ("x_per_thread", C.c_int), ("padded_x", C.c_int), ("padded_y", C.c_int),
                 ("padded_z", C.c_int), ("l2_bytes", C.c_double), ("corr_ms_last", C.c_double),
                 ("n_sms", C.c_int), ("engine_last", C.c_int), ("tc_available", C.c_int),
-                ("tc_variant_last", C.c_int), ("tc_ksteps_last", C.c_int)]
+                ("tc_variant_last", C.c_int), ("tc_ksteps_last", C.c_int),
+                ("tc_row_last", C.c_int), ("tc_rows_per_tile_last", C.c_int)]
 
 
 EXPORTS = ["dock_init", "dock_probe", "dock_probe_batch", "dock_score_grid", "dock_voxelize",

@@ -10,13 +10,16 @@ PKG = os.path.dirname(os.path.abspath(__file__))
 ROOT = os.path.dirname(PKG)
 CSRC = os.path.join(PKG, "csrc")
 LIB = os.path.join(PKG, "libdock.so")
-SOURCES = [os.path.join(CSRC, "dock.cu")]
-HEADERS = sorted(glob.glob(os.path.join(CSRC, "*.cuh"))) + [os.path.join(ROOT, "include", "dock.h")]
+# dock.cu = host logic + small kernels; launch_*.cu = one correlation-kernel family each (compiled in
+# parallel, then linked into one shared library)
+SOURCES = [os.path.join(CSRC, "dock.cu")] + sorted(glob.glob(os.path.join(CSRC, "launch_*.cu")))
+HEADERS = (sorted(glob.glob(os.path.join(CSRC, "*.cuh"))) + sorted(glob.glob(os.path.join(CSRC, "*.h"))) +
+           [os.path.join(ROOT, "include", "dock.h")])
 
 NVCC_FLAGS = [
     "-gencode", "arch=compute_100a,code=sm_100a",
     "-O3", "-lineinfo", "-std=c++17",
-    "-Xcompiler", "-fPIC", "-shared",
+    "-Xcompiler", "-fPIC",
     "-Xptxas", "-v",
 ]
 
@@ -38,16 +41,36 @@ def stale() -> bool:
 def build_native(force: bool = False, verbose: bool = False) -> str:
     if not force and not stale():
         return LIB
-    tmp = LIB + f".tmp{os.getpid()}"
-    cmd = [_nvcc(), *NVCC_FLAGS, "-I", os.path.join(ROOT, "include"), "-o", tmp, *SOURCES]
-    res = subprocess.run(cmd, capture_output=True, text=True)
+    from concurrent.futures import ThreadPoolExecutor
+    tag = f".tmp{os.getpid()}"
+    objs = [os.path.join(PKG, "build", os.path.basename(s) + tag + ".o") for s in SOURCES]
+    os.makedirs(os.path.join(PKG, "build"), exist_ok=True)
+
+    def compile_one(src_obj):
+        src, obj = src_obj
+        cmd = [_nvcc(), *NVCC_FLAGS, "-I", os.path.join(ROOT, "include"), "-c", "-o", obj, src]
+        return subprocess.run(cmd, capture_output=True, text=True)
+
+    with ThreadPoolExecutor(max_workers=max(1, min(len(SOURCES), os.cpu_count() or 1))) as ex:
+        results = list(ex.map(compile_one, zip(SOURCES, objs)))
+    log = ""
+    for src, res in zip(SOURCES, results):
+        log += f"== {os.path.basename(src)}\n" + res.stderr
+        if res.returncode != 0:
+            sys.stderr.write(res.stdout + res.stderr)
+            raise RuntimeError(f"nvcc failed compiling {os.path.basename(src)}")
+    tmp = LIB + tag
+    res = subprocess.run([_nvcc(), "-gencode", "arch=compute_100a,code=sm_100a", "-shared", "-o", tmp, *objs,
+                          "-lcuda"], capture_output=True, text=True)
     if res.returncode != 0:
         sys.stderr.write(res.stdout + res.stderr)
-        raise RuntimeError("nvcc failed building libdock.so")
+        raise RuntimeError("nvcc failed linking libdock.so")
+    for o in objs:
+        os.remove(o)
     if verbose:
-        sys.stderr.write(res.stderr)
+        sys.stderr.write(log)
     with open(os.path.join(PKG, "libdock.ptxas.txt"), "w") as f:
-        f.write(res.stderr)
+        f.write(log)
     os.replace(tmp, LIB)
     return LIB
 

@@ -20,7 +20,7 @@
 #include "dock.h"
 #include "dock_kernels.cuh"
 #include "dock_tc.cuh"
-#include "dock_tc_skew.cuh"
+#include "dock_launch.h"
 
 static_assert(sizeof(dock_pose) == 16, "dock_pose must be 16 bytes");
 static_assert(sizeof(dk::PoseOut) == sizeof(dock_pose), "kernel pose layout mismatch");
@@ -34,13 +34,12 @@ struct DevBuf {
     size_t cap = 0;
 };
 
-struct TcPlan {                // per-probe-size plan of the tcgen05 engine
+struct TcPlan {                // per-(variant, probe size) plan of the tcgen05 engine
     bool ok = false;
-    bool pair = false;         // PAIR scheme (one channel group): second receptor copy (Rhi(x), Rhi(x+1))
-    CUtensorMap tmap, tmap_pair;
-    int S1 = 0, S1p = 0, S2 = 0, S2p = 0;
-    int TXB = 0, TYB = 0, TZB = 0, box_bytes = 0, rec_stage_bytes = 0, n_rec_stages = 0, smem = 0, nsteps = 0,
-        wstages = 0;
+    CUtensorMap tmap, tmap_pair;   // (hi,lo) receptor copy and PAIR copy (Rhi(x), Rhi(x+1))
+    int ntt = 0, q = 0, ntx = 0, nty = 0, ntiles = 0;   // translations per row, rows per tile, tile counts
+    int S1 = 0, S1p = 0, S2 = 0, S2p = 0;                // variant 1: pass-1 / pass-2 K-steps (real, padded)
+    int box_bytes = 0, rec_stage_bytes = 0, n_rec_stages = 0, smem = 0, nsteps = 0, wstages = 0;
 };
 
 struct MPlan {                 // per-probe-size launch plan
@@ -69,14 +68,16 @@ struct dock_ctx {
     // tcgen05 engine
     int engine = 0;            // DOCK_TUNE_ENGINE: 0 auto, 1 FFMA, 2 tensor cores
     int engine_last = 0;
-    int tc_variant = 0;        // DOCK_TUNE_TC_VARIANT: 0 auto, 1 (Q4, 1 TMEM buffer), 2 (Q2, 2 buffers, CTA pair)
+    int tc_variant = 0;        // DOCK_TUNE_TC_VARIANT: 0 auto, 1 resident boxes (P <= 4), 2 streamed planes
     int tc_variant_last = 0;
-    int tc_ksteps_last = 0;
-    int tc_nepi = 0;          // epilogue warps (0 = one row per thread)   // K-steps (of 16) per translation row in the last tcgen05 launch
-    uint16_t* d_rec_tc = nullptr;
-    uint16_t* d_rec_pair = nullptr;   // PAIR-scheme receptor copy (P <= 4)
-    int tc_Gch = 0, tc_ntx = 0, tc_ntz = 0, tc_Xp = 0, tc_Yp = 0, tc_Zp = 0;
-    TcPlan tcplan[7][DOCK_MAX_M + 1];   // [variant][m]
+    int tc_m_last = 0;
+    int tc_ksteps_last = 0;    // K-steps (of 16) per translation row in the last tcgen05 launch
+    int tc_nepi = 0;           // epilogue warps (0 = 16)
+    uint16_t* d_rec_tc = nullptr;     // [g][Zp][Yp][Xp][8] bf16 (hi_0..3, lo_0..3)
+    uint16_t* d_rec_pair = nullptr;   // [g][Zp][Yp][Xp][8] bf16 (hi_0..3(X), hi_0..3(X+1))
+    int tc_Gch = 0, tc_Xp = 0, tc_Yp = 0, tc_Zp = 0;
+    int tcs_ntt = 128;         // variant 2 translations per MMA row, chosen for nx
+    TcPlan tcplan[3][DOCK_MAX_M + 1];   // [variant][m]
     DevBuf Wtc;
     // diagnostics (environment, read at init): DOCK_TC_TRACE=1 prints per-role cycle counters of every
     // k_corr_tc launch to stderr; DOCK_TC_DEBUG=1|2 disables parts of the epilogue (timing only)
@@ -252,246 +253,80 @@ dock_status make_plan(dock_ctx* ctx, int m)
     return DOCK_OK;
 }
 
-template <int M, bool GRID>
-cudaError_t launch_corr_t(const MPlan& pl, const dk::CorrArgs& a, int grid, cudaStream_t st)
-{
-    auto kern = dk::k_corr<M, GRID>;
-    cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, pl.smem);
-    if (e != cudaSuccess) return e;
-    kern<<<grid, dk::NTHREADS, pl.smem, st>>>(pl.tmap, a);
-    return cudaGetLastError();
-}
-
-template <bool GRID>
-cudaError_t launch_corr(int m, const MPlan& pl, const dk::CorrArgs& a, int grid, cudaStream_t st)
-{
-    switch (m) {
-        case 1: return launch_corr_t<1, GRID>(pl, a, grid, st);
-        case 2: return launch_corr_t<2, GRID>(pl, a, grid, st);
-        case 3: return launch_corr_t<3, GRID>(pl, a, grid, st);
-        case 4: return launch_corr_t<4, GRID>(pl, a, grid, st);
-        case 5: return launch_corr_t<5, GRID>(pl, a, grid, st);
-        case 6: return launch_corr_t<6, GRID>(pl, a, grid, st);
-        case 7: return launch_corr_t<7, GRID>(pl, a, grid, st);
-        case 8: return launch_corr_t<8, GRID>(pl, a, grid, st);
-        default: return cudaErrorInvalidValue;
-    }
-}
-
-int tc_txb(int m) { return tc::NT + (m + 1) / 2 * 2 - 1; }
-// tcgen05 variants: 1 = Q4 rows x 1 TMEM buffer, single CTA; 2 = Q2 rows x 2 buffers, CTA pair + multicast;
-// 3 = cta_group::2 (4 rows over a CTA pair); 4 = Q2 x 2 buffers, single CTA; 5 / 6 = the row-skewed schedule
-// (dock_tc_skew.cuh) with Q4 x 1 buffer / Q2 x 2 buffers and z-plane receptor staging.
-// tile rows (translation rows per tile): variants 1, 3 and 5 tile 4 rows, the others 2
-inline int tc_q(int v) { return (v == 2 || v == 4 || v == 6) ? 2 : 4; }
-inline int tc_cl(int v) { return (v == 2 || v == 3) ? 2 : 1; }
-inline bool tc_skew(int v) { return v == 5 || v == 6; }
-// receptor rows held per CTA (variant 3 splits the 4 tile rows over the CTA pair)
-inline int tc_rows_cta(int v) { return v == 3 ? 2 : tc_q(v); }
-inline int tc_nty(const dock_ctx* c, int v) { return (c->ny + tc_q(v) - 1) / tc_q(v); }
-inline int tc_ntiles(const dock_ctx* c, int v) { return c->tc_ntx * tc_nty(c, v) * c->tc_ntz; }
-
-int tc_txb_any(int m) { return std::max(tc_txb(m), 4 * ((m + 3) / 4) + 126); }
-
+// tcgen05 engine (dock_tc.cuh): variant 1 = one channel group, both receptor boxes resident, 128
+// translations x 4 rows per tile; variant 2 = any channel count, receptor streamed one (group, z-plane)
+// unit at a time, NTT in {64, 128, 160} translations per row (chosen at init for nx) x tcs_q(NTT) rows.
 dock_status make_tc_plan(dock_ctx* ctx, int m, int v)
 {
     TcPlan& pl = ctx->tcplan[v][m];
-    if (pl.ok || !ctx->d_rec_tc) return DOCK_OK;
+    if (pl.ok || !ctx->d_rec_tc || !ctx->d_rec_pair) return DOCK_OK;
     const int KS = tc::KSTEPS;
     const int budget = kSmemLimit - 2048;   // static shared memory (barriers) and slack
     const int stage = KS * tc::WCHUNK;
-    const int min_ring = 2 * stage;
-    // PAIR needs the (hi,lo) box and the (hi,hi') box resident together; otherwise the 2-pass scheme
-    const int pair_box = round_up(16 * tc_txb_any(m) * (tc_rows_cta(v) + m - 1) * m, 1024);
-    pl.pair = ctx->tc_Gch == 1 && ctx->d_rec_pair != nullptr && 2 * pair_box + min_ring <= budget;
-    if (!pl.pair && v != 1) return DOCK_OK;          // variants 2-6 are built for the PAIR scheme only
-    if (tc_skew(v) && m < 3) return DOCK_OK;        // the skewed schedule needs >= Q weight stages per tile
-    pl.TXB = pl.pair ? tc_txb_any(m) : tc_txb(m);
-    pl.TYB = tc_rows_cta(v) + m - 1;
-    pl.TZB = m;
-    pl.box_bytes = 16 * pl.TXB * pl.TYB * pl.TZB;
-    // the single-CTA PAIR kernels bake the box geometry into their descriptor offsets
-    if (pl.pair && tc_cl(v) == 1 && (pl.TXB != tc::pair_txb(m) || pl.TYB != tc_q(v) + m - 1))
-        return fail(ctx, DOCK_E_CUDA, "tcgen05 PAIR box geometry mismatch");
-    pl.rec_stage_bytes = round_up(ctx->tc_Gch * pl.box_bytes, 1024);
-    if (tc_skew(v)) pl.rec_stage_bytes = round_up(m * (int)tc::plane_stride(m, tc_q(v)), 1024);
-    if (pl.pair) {
-        pl.S1 = m * m * ((m + 1) / 2);
+    int TXB = 0, TYB = 0, TZB = 0;
+    if (v == 1) {
+        if (ctx->tc_Gch != 1) return DOCK_OK;   // one channel group only
+        pl.ntt = tc::NT;
+        pl.q = 4;
+        TXB = tc::pair_txb(m, pl.ntt);
+        TYB = pl.q + m - 1;
+        TZB = m;
+        pl.box_bytes = 16 * TXB * TYB * TZB;
+        pl.rec_stage_bytes = round_up(pl.box_bytes, 1024);
+        pl.n_rec_stages = 2;   // main box + pair box
+        const int MXP = (m + 1) / 2, MXQ = (m + 3) / 4;
+        pl.S1 = m * m * MXP;
         pl.S1p = round_up(pl.S1, KS);
-        pl.S2 = m * m * ((m + 3) / 4);
+        pl.S2 = m * m * MXQ;
         pl.S2p = round_up(pl.S2, KS);
         pl.nsteps = pl.S1p + pl.S2p;
+        if (2 * pl.rec_stage_bytes + 3 * stage > budget) return DOCK_OK;   // not eligible for this m
     } else {
-        pl.nsteps = ctx->tc_Gch * 2 * m * m * ((m + 1) / 2);
-        if (pl.nsteps % KS) return DOCK_OK;   // the 2-pass scheme needs whole ring stages
+        pl.ntt = ctx->tcs_ntt;
+        pl.q = tcs_q(pl.ntt);
+        TXB = tc::pair_txb(m, pl.ntt);
+        TYB = pl.q + m - 1;
+        TZB = 1;
+        pl.box_bytes = 16 * TXB * TYB;   // one z-plane
+        pl.rec_stage_bytes = round_up(2 * (int)tc::stream_plane_stride(m, pl.ntt, pl.q), 1024);
+        pl.n_rec_stages = 3 * pl.rec_stage_bytes + 6 * stage <= budget ? 3 : 2;
+        if (pl.n_rec_stages * pl.rec_stage_bytes + 3 * stage > budget) return DOCK_OK;
+        pl.nsteps = ctx->tc_Gch * m * tc::unit_ksteps_padded(m);
     }
-    if (2 * pl.rec_stage_bytes + min_ring <= budget) pl.n_rec_stages = 2;
-    else if (!pl.pair && pl.rec_stage_bytes + min_ring <= budget) pl.n_rec_stages = 1;
-    else return DOCK_OK;                    // this m is not eligible for the tensor-core engine
+    if (TXB > 256 || TYB > 256) return DOCK_OK;   // TMA box limit
+    pl.ntx = (ctx->nx + pl.ntt - 1) / pl.ntt;
+    pl.nty = (ctx->ny + pl.q - 1) / pl.q;
+    pl.ntiles = pl.ntx * pl.nty * ctx->nz;
+    if ((pl.ntx - 1) * pl.ntt + TXB > ctx->tc_Xp || pl.nty * pl.q + m - 1 > ctx->tc_Yp)
+        return fail(ctx, DOCK_E_CUDA, "tcgen05 receptor padding too small");
     pl.wstages = std::min(tc::WSTAGES, (budget - pl.n_rec_stages * pl.rec_stage_bytes) / stage);
-    if (tc_skew(v) && pl.wstages < tc_q(v) + 1) return DOCK_OK;   // every row holds one stage of the ring
-    const int ring = pl.wstages * stage;
     // >= 116 KB keeps one CTA per SM: every CTA allocates all 512 TMEM columns
-    pl.smem = std::max(pl.n_rec_stages * pl.rec_stage_bytes + ring, 116 * 1024);
+    pl.smem = std::max(pl.n_rec_stages * pl.rec_stage_bytes + pl.wstages * stage, 116 * 1024);
     auto fn = encode_fn();
     if (!fn) return fail(ctx, DOCK_E_CUDA, "cuTensorMapEncodeTiled unavailable");
     const cuuint64_t X = ctx->tc_Xp, Y = ctx->tc_Yp, Z = ctx->tc_Zp;
     cuuint64_t dims[5] = {8, X, Y, Z, (cuuint64_t)ctx->tc_Gch};
     cuuint64_t strides[4] = {16, X * 16, X * Y * 16, X * Y * Z * 16};
-    // the skewed kernels stage the receptor one z-plane per TMA box
-    cuuint32_t box[5] = {8, (cuuint32_t)pl.TXB, (cuuint32_t)pl.TYB, (cuuint32_t)(tc_skew(v) ? 1 : pl.TZB), 1};
+    cuuint32_t box[5] = {8, (cuuint32_t)TXB, (cuuint32_t)TYB, (cuuint32_t)TZB, 1};
     cuuint32_t es[5] = {1, 1, 1, 1, 1};
-    for (int which = 0; which < (pl.pair ? 2 : 1); which++) {
+    for (int which = 0; which < 2; which++) {
         CUresult r = fn(which ? &pl.tmap_pair : &pl.tmap, CU_TENSOR_MAP_DATA_TYPE_BFLOAT16, 5,
                         which ? (void*)ctx->d_rec_pair : (void*)ctx->d_rec_tc, dims, strides, box, es,
                         CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_L2_256B,
                         CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
         if (r != CUDA_SUCCESS) return fail(ctx, DOCK_E_CUDA, "cuTensorMapEncodeTiled (bf16) failed (%d)", (int)r);
     }
-    if (!pl.pair) pl.tmap_pair = pl.tmap;
     pl.ok = true;
     return DOCK_OK;
 }
 
-template <int M, int Q, int NBUF, int CL, bool PAIR, bool GRID>
-cudaError_t launch_tc_t(const TcPlan& pl, const tc::TcArgs& a, int grid, cudaStream_t st)
+cudaError_t launch_tc(int m, int v, bool grid, const TcPlan& pl, const tc::TcArgs& a, int nblocks, cudaStream_t st)
 {
-    auto kern = tc::k_corr_tc<M, Q, NBUF, CL, PAIR, GRID>;
-    cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, pl.smem);
-    if (e != cudaSuccess) return e;
-    if constexpr (CL == 1) {
-        kern<<<grid, (2 + a.nepi) * 32, pl.smem, st>>>(pl.tmap, pl.tmap_pair, a);
-    } else {
-        cudaLaunchConfig_t cfg{};
-        cfg.gridDim = dim3(grid);
-        cfg.blockDim = dim3((2 + a.nepi) * 32);
-        cfg.dynamicSmemBytes = pl.smem;
-        cfg.stream = st;
-        cudaLaunchAttribute at[1];
-        at[0].id = cudaLaunchAttributeClusterDimension;
-        at[0].val.clusterDim.x = CL;
-        at[0].val.clusterDim.y = 1;
-        at[0].val.clusterDim.z = 1;
-        cfg.attrs = at;
-        cfg.numAttrs = 1;
-        e = cudaLaunchKernelEx(&cfg, kern, pl.tmap, pl.tmap_pair, a);
-        if (e != cudaSuccess) return e;
-    }
-    return cudaGetLastError();
+    if (v == 1) return dock_launch_tc1(m, grid, pl.tmap, pl.tmap_pair, pl.smem, a, nblocks, st);
+    return dock_launch_tcs(m, pl.ntt, grid, pl.tmap, pl.tmap_pair, pl.smem, a, nblocks, st);
 }
 
-template <int V, bool PAIR, bool GRID>
-cudaError_t launch_tc_v(int m, const TcPlan& pl, const tc::TcArgs& a, int grid, cudaStream_t st)
-{
-    constexpr int Q = V == 1 ? 4 : 2, NB = V == 1 ? 1 : 2, CL = (V == 1 || V == 4) ? 1 : 2;
-    switch (m) {
-        case 1: return launch_tc_t<1, Q, NB, CL, PAIR, GRID>(pl, a, grid, st);
-        case 2: return launch_tc_t<2, Q, NB, CL, PAIR, GRID>(pl, a, grid, st);
-        case 3: return launch_tc_t<3, Q, NB, CL, PAIR, GRID>(pl, a, grid, st);
-        case 4: return launch_tc_t<4, Q, NB, CL, PAIR, GRID>(pl, a, grid, st);
-        case 5: return launch_tc_t<5, Q, NB, CL, PAIR, GRID>(pl, a, grid, st);
-        case 6: return launch_tc_t<6, Q, NB, CL, PAIR, GRID>(pl, a, grid, st);
-        case 7: return launch_tc_t<7, Q, NB, CL, PAIR, GRID>(pl, a, grid, st);
-        case 8: return launch_tc_t<8, Q, NB, CL, PAIR, GRID>(pl, a, grid, st);
-        default: return cudaErrorInvalidValue;
-    }
-}
-
-template <int M, bool GRID>
-cudaError_t launch_tc2_t(const TcPlan& pl, const tc::TcArgs& a, int grid, cudaStream_t st)
-{
-    auto kern = tc::k_corr_tc2<M, GRID>;
-    cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, pl.smem);
-    if (e != cudaSuccess) return e;
-    cudaLaunchConfig_t cfg{};
-    cfg.gridDim = dim3(grid);
-    cfg.blockDim = dim3((2 + a.nepi) * 32);
-    cfg.dynamicSmemBytes = pl.smem;
-    cfg.stream = st;
-    cudaLaunchAttribute at[1];
-    at[0].id = cudaLaunchAttributeClusterDimension;
-    at[0].val.clusterDim.x = 2;
-    at[0].val.clusterDim.y = 1;
-    at[0].val.clusterDim.z = 1;
-    cfg.attrs = at;
-    cfg.numAttrs = 1;
-    e = cudaLaunchKernelEx(&cfg, kern, pl.tmap, pl.tmap_pair, a);
-    if (e != cudaSuccess) return e;
-    return cudaGetLastError();
-}
-
-template <bool GRID>
-cudaError_t launch_tc2(int m, const TcPlan& pl, const tc::TcArgs& a, int grid, cudaStream_t st)
-{
-    switch (m) {
-        case 1: return launch_tc2_t<1, GRID>(pl, a, grid, st);
-        case 2: return launch_tc2_t<2, GRID>(pl, a, grid, st);
-        case 3: return launch_tc2_t<3, GRID>(pl, a, grid, st);
-        case 4: return launch_tc2_t<4, GRID>(pl, a, grid, st);
-        case 5: return launch_tc2_t<5, GRID>(pl, a, grid, st);
-        case 6: return launch_tc2_t<6, GRID>(pl, a, grid, st);
-        case 7: return launch_tc2_t<7, GRID>(pl, a, grid, st);
-        case 8: return launch_tc2_t<8, GRID>(pl, a, grid, st);
-        default: return cudaErrorInvalidValue;
-    }
-}
-
-template <int M, int Q, int NBUF, bool GRID>
-cudaError_t launch_skew_t(const TcPlan& pl, const tc::TcArgs& a, int grid, cudaStream_t st)
-{
-    auto kern = tc::k_corr_tc_skew<M, Q, NBUF, GRID>;
-    cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, pl.smem);
-    if (e != cudaSuccess) return e;
-    kern<<<grid, (2 + a.nepi) * 32, pl.smem, st>>>(pl.tmap, pl.tmap_pair, a);
-    return cudaGetLastError();
-}
-
-template <int Q, int NBUF, bool GRID>
-cudaError_t launch_skew(int m, const TcPlan& pl, const tc::TcArgs& a, int grid, cudaStream_t st)
-{
-    switch (m) {
-        case 3: return launch_skew_t<3, Q, NBUF, GRID>(pl, a, grid, st);
-        case 4: return launch_skew_t<4, Q, NBUF, GRID>(pl, a, grid, st);
-        case 5: return launch_skew_t<5, Q, NBUF, GRID>(pl, a, grid, st);
-        case 6: return launch_skew_t<6, Q, NBUF, GRID>(pl, a, grid, st);
-        case 7: return launch_skew_t<7, Q, NBUF, GRID>(pl, a, grid, st);
-        case 8: return launch_skew_t<8, Q, NBUF, GRID>(pl, a, grid, st);
-        default: return cudaErrorInvalidValue;
-    }
-}
-
-template <bool GRID>
-cudaError_t launch_tc(int m, int v, const TcPlan& pl, const tc::TcArgs& a, int grid, cudaStream_t st)
-{
-    if (v == 5) return launch_skew<4, 1, GRID>(m, pl, a, grid, st);
-    if (v == 6) return launch_skew<2, 2, GRID>(m, pl, a, grid, st);
-    if (v == 3) return launch_tc2<GRID>(m, pl, a, grid, st);
-    if (!pl.pair) return v == 1 ? launch_tc_v<1, false, GRID>(m, pl, a, grid, st) : cudaErrorInvalidValue;
-    if (v == 4) return launch_tc_v<4, true, GRID>(m, pl, a, grid, st);
-    return v == 1 ? launch_tc_v<1, true, GRID>(m, pl, a, grid, st) : launch_tc_v<2, true, GRID>(m, pl, a, grid, st);
-}
-
-// Regions for the CTA-pair variant: an even number that divides the tiles (equal tile counts per pair).
-int choose_regions_pair(const dock_ctx* ctx, int64_t n_blocks, int nt)
-{
-    int best = 0;
-    double best_cost = 1e300;
-    for (int G = 2; G <= std::min(nt, 1024); G += 2) {
-        if (nt % G) continue;
-        if (ctx->regions_override > 0 && G != ctx->regions_override) continue;
-        const int tpr = nt / G;
-        const int64_t items = n_blocks * G;
-        const int64_t waves = (items + ctx->n_sms - 1) / ctx->n_sms;
-        const double cost = double(waves) * (tpr + 0.5);
-        if (cost < best_cost - 1e-9) {
-            best_cost = cost;
-            best = G;
-        }
-    }
-    return best;
-}
-
-// Regions per item for a given number of rotation batches and tiles.
+// Regions per rotation block (tcgen05): minimise waves * (tiles per item + per-item overhead).
 int choose_regions_n(const dock_ctx* ctx, int64_t n_batches, int nt)
 {
     if (ctx->regions_override > 0) return std::min(ctx->regions_override, nt);
@@ -688,7 +523,7 @@ dock_status run_grid(dock_ctx* ctx, int m, int n_slots, const float* Lw, float* 
     int G = choose_regions(ctx, nb);
     dk::CorrArgs a = corr_args(ctx, m, n_slots, G, Lw);
     a.grid = grid;
-    CU(launch_corr<true>(m, ctx->plan[m], a, (int)(nb * G), ctx->stream));
+    CU(dock_launch_ffma(m, true, ctx->plan[m].tmap, ctx->plan[m].smem, a, (int)(nb * G), ctx->stream));
     ctx->kernels_last++;
     return DOCK_OK;
 }
@@ -758,70 +593,42 @@ tc::TcArgs tc_args(dock_ctx* ctx, int m, int v, int n_slots, int G, const unsign
     a.nx = ctx->nx;
     a.ny = ctx->ny;
     a.nz = ctx->nz;
-    a.ntx = ctx->tc_ntx;
-    a.nty = tc_nty(ctx, v);
-    a.ntz = ctx->tc_ntz;
-    a.ntiles = tc_ntiles(ctx, v);
+    a.ntx = tp.ntx;
+    a.nty = tp.nty;
+    a.ntz = ctx->nz;
+    a.ntiles = tp.ntiles;
     a.G_ch = ctx->tc_Gch;
     a.n_slots = n_slots;
     a.G = G;
     a.tiles_per_region = (a.ntiles + G - 1) / G;
     a.nsteps = tp.nsteps;
     a.W = W;
-    a.TXB = tp.TXB;
-    a.TYB = tp.TYB;
-    a.TZB = tp.TZB;
     a.box_bytes = tp.box_bytes;
     a.rec_stage_bytes = tp.rec_stage_bytes;
     a.n_rec_stages = tp.n_rec_stages;
     a.wstages = tp.wstages;
-    a.nepi = ctx->tc_nepi > 0 ? std::min(16, ctx->tc_nepi) : ((v == 2 || v == 4) ? 8 : 16);   // one row per thread
+    a.nepi = ctx->tc_nepi > 0 ? std::min(16, ctx->tc_nepi) : 16;
     a.trace = ctx->d_trace;
     a.dbg = ctx->tc_dbg;
-    a.S1 = tp.S1;
-    a.S1p = tp.S1p;
-    a.S2 = tp.S2;
-    a.S2p = tp.S2p;
     return a;
 }
 
 // Variant + regions for a launch over n_slots rotations; returns false if the tensor cores can't run m.
+// Auto: variant 1 where it runs with the same row width as variant 2 would use (its resident boxes
+// need no per-plane synchronisation), else variant 2.
 bool plan_tc_launch(dock_ctx* ctx, int m, int n_slots, int* v_out, int* G_out)
 {
     const int64_t n_blocks = (n_slots + tc::ROT - 1) / tc::ROT;
-    const bool ok2 = ctx->tcplan[2][m].ok, ok1 = ctx->tcplan[1][m].ok;
-    // variant 1 is the default (fastest measured); variant 2 only when asked for and possible
-    // (it needs an even region count dividing the tiles)
-    if (ctx->tc_variant == 2 && ok2) {
-        const int G = choose_regions_pair(ctx, n_blocks, tc_ntiles(ctx, 2));
-        if (G > 0) {
-            *v_out = 2;
-            *G_out = G;
-            return true;
-        }
-    }
-    for (int v : {4, 5, 6}) {
-        if (ctx->tc_variant == v && ctx->tcplan[v][m].ok) {
-            *v_out = v;
-            *G_out = choose_regions_n(ctx, n_blocks, tc_ntiles(ctx, v));
-            return true;
-        }
-    }
-    if (ctx->tc_variant == 3 && ctx->tcplan[3][m].ok) {
-        // CTA pairs over pairs of rotation blocks; a pair occupies two SMs
-        const int64_t n_pairs = (n_blocks + 1) / 2;
-        dock_ctx tmp = *ctx;
-        tmp.n_sms = ctx->n_sms / 2;
-        *v_out = 3;
-        *G_out = choose_regions_n(&tmp, n_pairs, tc_ntiles(ctx, 3));
-        return true;
-    }
-    if (ok1) {
-        *v_out = 1;
-        *G_out = choose_regions_n(ctx, n_blocks, tc_ntiles(ctx, 1));
-        return true;
-    }
-    return false;
+    const bool ok1 = ctx->tcplan[1][m].ok, ok2 = ctx->tcplan[2][m].ok;
+    int v = 0;
+    if (ctx->tc_variant == 1 && ok1) v = 1;
+    else if (ctx->tc_variant == 2 && ok2) v = 2;
+    else if (ok1 && (ctx->tcs_ntt == tc::NT || !ok2)) v = 1;
+    else if (ok2) v = 2;
+    if (!v) return false;
+    *v_out = v;
+    *G_out = choose_regions_n(ctx, n_blocks, ctx->tcplan[v][m].ntiles);
+    return true;
 }
 
 // Engine choice: tensor cores when a plan for this m exists (auto) or when forced.
@@ -836,19 +643,20 @@ dock_status select_engine(dock_ctx* ctx, int m, bool* use_tc)
     return DOCK_OK;
 }
 
-// Pack folded FP32 weights into the tcgen05 A-operand layout of plan tp.
-dock_status pack_weights_tc(dock_ctx* ctx, int m, const TcPlan& tp, int n_slots, const float* Lw)
+// Pack folded FP32 weights into the tcgen05 A-operand layout of variant v.
+dock_status pack_weights_tc(dock_ctx* ctx, int m, int v, int n_slots, const float* Lw)
 {
+    const TcPlan& tp = ctx->tcplan[v][m];
     const int64_t n_blocks = (n_slots + tc::ROT - 1) / tc::ROT;
     TRY(ensure(ctx, ctx->Wtc, (size_t)n_blocks * tp.nsteps * tc::WCHUNK));
     const int64_t rows = n_blocks * tp.nsteps * 2 * tc::ROT;
     const int grid = (int)std::min<int64_t>((rows + 255) / 256, 65535);
     unsigned char* W = static_cast<unsigned char*>(ctx->Wtc.p);
-    if (tp.pair)
+    if (v == 1)
         tc::k_pack_weights_tc_pair<<<grid, 256, 0, ctx->stream>>>(Lw, W, n_slots, ctx->P, m, tp.S1, tp.S1p, tp.S2,
                                                                    tp.S2p);
     else
-        tc::k_pack_weights_tc<<<grid, 256, 0, ctx->stream>>>(Lw, W, n_slots, ctx->P, ctx->tc_Gch, m, tp.nsteps);
+        tc::k_pack_weights_tcs<<<grid, 256, 0, ctx->stream>>>(Lw, W, n_slots, ctx->P, m, tp.nsteps);
     CU(cudaGetLastError());
     ctx->kernels_last++;
     return DOCK_OK;
@@ -860,11 +668,11 @@ dock_status run_grid_tc(dock_ctx* ctx, int m, int n_slots, const float* Lw, floa
     const int64_t n_blocks = (n_slots + tc::ROT - 1) / tc::ROT;
     int v = 0, G = 0;
     if (!plan_tc_launch(ctx, m, n_slots, &v, &G)) return fail(ctx, DOCK_E_UNSUPPORTED, "no tensor-core plan");
-    TRY(pack_weights_tc(ctx, m, ctx->tcplan[v][m], n_slots, Lw));
+    TRY(pack_weights_tc(ctx, m, v, n_slots, Lw));
     tc::TcArgs a = tc_args(ctx, m, v, n_slots, G, static_cast<const unsigned char*>(ctx->Wtc.p));
     a.grid = grid;
-    const int64_t items = v == 3 ? 2 * ((n_blocks + 1) / 2) * G : n_blocks * G;
-    CU(launch_tc<true>(m, v, ctx->tcplan[v][m], a, (int)items, ctx->stream));
+    const int64_t items = n_blocks * G;
+    CU(launch_tc(m, v, true, ctx->tcplan[v][m], a, (int)items, ctx->stream));
     ctx->kernels_last++;
     return DOCK_OK;
 }
@@ -1020,33 +828,39 @@ dock_status dock_init(const dock_grid_desc* g, const float* receptor, const floa
     }
     dk::k_pad_receptor<<<2048, 256, 0, ctx->stream>>>(d_src, ctx->d_rec, ctx->nx, ctx->ny, ctx->nz, G.Xp, G.Yp,
                                                        G.Zp, P);
-    // tcgen05 engine: bf16-split, channel-grouped, cyclic-halo copy of the receptor
+    // tcgen05 engine: bf16-split, channel-grouped, cyclic-halo copies of the receptor
     {
         ctx->tc_Gch = (P + 3) / 4;
-        ctx->tc_ntx = (ctx->nx + tc::NT - 1) / tc::NT;
-        ctx->tc_ntz = ctx->nz;
-        int txb_max = 0;
-        for (int mm = 1; mm <= ctx->m_max; mm++) txb_max = std::max(txb_max, tc_txb_any(mm));
-        ctx->tc_Xp = round_up((ctx->tc_ntx - 1) * tc::NT + txb_max, 2);
-        ctx->tc_Yp = round_up(ctx->ny, 4) + ctx->m_max - 1;   // covers Q = 4 and Q = 2 tilings
+        // variant 2 row width: the fewest wasted x translations (ties: 128, then 160, then 64)
+        int best_w = 1 << 30;
+        for (int ntt : {128, 160, 64}) {
+            const int w = (ctx->nx + ntt - 1) / ntt * ntt;
+            if (w < best_w) {
+                best_w = w;
+                ctx->tcs_ntt = ntt;
+            }
+        }
+        const int q2 = tcs_q(ctx->tcs_ntt);
+        const int ntx1 = (ctx->nx + tc::NT - 1) / tc::NT, ntx2 = (ctx->nx + ctx->tcs_ntt - 1) / ctx->tcs_ntt;
+        int xp = 0;
+        for (int mm = 1; mm <= ctx->m_max; mm++)
+            xp = std::max({xp, (ntx1 - 1) * tc::NT + tc::pair_txb(mm, tc::NT),
+                           (ntx2 - 1) * ctx->tcs_ntt + tc::pair_txb(mm, ctx->tcs_ntt)});
+        ctx->tc_Xp = round_up(xp, 2);
+        ctx->tc_Yp = std::max(round_up(ctx->ny, 4), round_up(ctx->ny, q2)) + ctx->m_max - 1;
         ctx->tc_Zp = ctx->nz + ctx->m_max - 1;
         const size_t bytes = (size_t)ctx->tc_Gch * ctx->tc_Zp * ctx->tc_Yp * ctx->tc_Xp * 16;
-        if (cudaMalloc(&ctx->d_rec_tc, bytes) == cudaSuccess) {
+        if (cudaMalloc(&ctx->d_rec_tc, bytes) == cudaSuccess && cudaMalloc(&ctx->d_rec_pair, bytes) == cudaSuccess) {
             tc::k_pack_receptor_tc<<<2048, 256, 0, ctx->stream>>>(d_src, ctx->d_rec_tc, ctx->nx, ctx->ny, ctx->nz,
                                                                    ctx->tc_Xp, ctx->tc_Yp, ctx->tc_Zp, P, ctx->tc_Gch);
-            if (ctx->tc_Gch == 1) {
-                const size_t pbytes = (size_t)ctx->tc_Zp * ctx->tc_Yp * ctx->tc_Xp * 16;
-                if (cudaMalloc(&ctx->d_rec_pair, pbytes) == cudaSuccess) {
-                    tc::k_pack_receptor_pair_tc<<<2048, 256, 0, ctx->stream>>>(
-                        d_src, ctx->d_rec_pair, ctx->nx, ctx->ny, ctx->nz, ctx->tc_Xp, ctx->tc_Yp, ctx->tc_Zp, P);
-                } else {
-                    cudaGetLastError();
-                    ctx->d_rec_pair = nullptr;
-                }
-            }
+            tc::k_pack_receptor_pair_tc<<<2048, 256, 0, ctx->stream>>>(d_src, ctx->d_rec_pair, ctx->nx, ctx->ny,
+                                                                        ctx->nz, ctx->tc_Xp, ctx->tc_Yp, ctx->tc_Zp, P,
+                                                                        ctx->tc_Gch);
         } else {
             cudaGetLastError();
+            cudaFree(ctx->d_rec_tc);
             ctx->d_rec_tc = nullptr;   // the tensor-core engine is then unavailable
+            ctx->d_rec_pair = nullptr;
         }
     }
     cudaError_t e = cudaGetLastError();
@@ -1058,7 +872,7 @@ dock_status dock_init(const dock_grid_desc* g, const float* receptor, const floa
     for (int m = 1; m <= ctx->m_max; m++) {
         dock_status s = make_plan(ctx, m);
         if (s != DOCK_OK && m == ctx->m_max) return bail(s);
-        for (int v = 1; v <= 6; v++)
+        for (int v = 1; v <= 2; v++)
             if (make_tc_plan(ctx, m, v) != DOCK_OK) return bail(DOCK_E_CUDA);
     }
     *out = ctx;
@@ -1079,7 +893,7 @@ dock_status dock_set_tuning(dock_ctx* ctx, int key, int64_t value)
             ctx->engine = (int)value;
             return DOCK_OK;
         case DOCK_TUNE_TC_VARIANT:
-            if (value < 0 || value > 6) return fail(ctx, DOCK_E_INVALID_ARG, "tc variant must be 0..6");
+            if (value < 0 || value > 2) return fail(ctx, DOCK_E_INVALID_ARG, "tc variant must be 0, 1 or 2");
             ctx->tc_variant = (int)value;
             return DOCK_OK;
         case DOCK_TUNE_TC_EPILOGUE_WARPS:
@@ -1129,6 +943,11 @@ dock_status dock_get_info(const dock_ctx* ctx, dock_info* info)
     info->tc_available = (ctx->tcplan[1][ctx->m_max].ok || ctx->tcplan[2][ctx->m_max].ok) ? 1 : 0;
     info->tc_variant_last = ctx->tc_variant_last;
     info->tc_ksteps_last = ctx->tc_ksteps_last;
+    if (ctx->tc_variant_last > 0) {
+        const TcPlan& tp = ctx->tcplan[ctx->tc_variant_last][ctx->tc_m_last];
+        info->tc_row_last = tp.ntt;
+        info->tc_rows_per_tile_last = tp.q;
+    }
     return DOCK_OK;
 }
 
@@ -1206,9 +1025,10 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
         const int64_t n_blocks = (n_units + tc::ROT - 1) / tc::ROT;
         int v = 0, G = 0;
         if (!plan_tc_launch(ctx, m, n_units, &v, &G)) return fail(ctx, DOCK_E_UNSUPPORTED, "no tensor-core plan");
-        TRY(pack_weights_tc(ctx, m, ctx->tcplan[v][m], n_units, static_cast<const float*>(ctx->Lw.p)));
+        TRY(pack_weights_tc(ctx, m, v, n_units, static_cast<const float*>(ctx->Lw.p)));
         ctx->tc_variant_last = v;
         ctx->tc_ksteps_last = ctx->tcplan[v][m].nsteps;
+        ctx->tc_m_last = m;
         tc::TcArgs ta = tc_args(ctx, m, v, n_units, G, static_cast<const unsigned char*>(ctx->Wtc.p));
         ta.k = k;
         ta.rho = rho;
@@ -1217,11 +1037,11 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
         ta.mu = mup;
         ta.cnt = cntp;
         ta.cand = candp;
-        const int64_t items = v == 3 ? 2 * ((n_blocks + 1) / 2) * G : n_blocks * G;
+        const int64_t items = n_blocks * G;
         if (items > 0x7fffffff) return fail(ctx, DOCK_E_UNSUPPORTED, "too many work items");
         if (ctx->d_trace) CU(cudaMemsetAsync(ctx->d_trace, 0, sizeof(unsigned long long) * tc::TR_N, ctx->stream));
         CU(cudaEventRecord(ctx->ev_corr[0], ctx->stream));
-        CU(launch_tc<false>(m, v, ctx->tcplan[v][m], ta, (int)items, ctx->stream));
+        CU(launch_tc(m, v, false, ctx->tcplan[v][m], ta, (int)items, ctx->stream));
         CU(cudaEventRecord(ctx->ev_corr[1], ctx->stream));
         if (ctx->d_trace) {
             unsigned long long h[tc::TR_N];
@@ -1255,7 +1075,7 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
         const int64_t items = n_batches * G;
         if (items > 0x7fffffff) return fail(ctx, DOCK_E_UNSUPPORTED, "too many work items");
         CU(cudaEventRecord(ctx->ev_corr[0], ctx->stream));
-        CU(launch_corr<false>(m, ctx->plan[m], a, (int)items, ctx->stream));
+        CU(dock_launch_ffma(m, false, ctx->plan[m].tmap, ctx->plan[m].smem, a, (int)items, ctx->stream));
         CU(cudaEventRecord(ctx->ev_corr[1], ctx->stream));
         ctx->regions_last = G;
         ctx->items_last = items;

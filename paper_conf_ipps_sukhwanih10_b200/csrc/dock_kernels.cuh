@@ -204,6 +204,7 @@ __device__ __forceinline__ void prefetch_tmap(const CUtensorMap* map)
 // ------------------------------------------------------------------ a0: cyclic-halo padding
 
 // Rpad[p][Z][Y][X] = R[p][Z mod nz][Y mod ny][X mod nx]   (reading Q2: cyclic translations)
+#ifndef DOCK_LAUNCHER_TU   // defined once, in dock.cu
 __global__ void k_pad_receptor(const float* __restrict__ R, float* __restrict__ Rp, int nx, int ny, int nz,
                                int Xp, int Yp, int Zp, int P)
 {
@@ -219,7 +220,9 @@ __global__ void k_pad_receptor(const float* __restrict__ R, float* __restrict__ 
         Rp[i] = R[((static_cast<size_t>(p) * nz + Z % nz) * ny + Y % ny) * nx + X % nx];
     }
 }
+#endif
 
+#ifndef DOCK_LAUNCHER_TU   // defined once, in dock.cu
 __global__ void k_count_nonfinite(const float* __restrict__ a, size_t n, unsigned int* bad)
 {
     unsigned c = 0;
@@ -228,6 +231,7 @@ __global__ void k_count_nonfinite(const float* __restrict__ a, size_t n, unsigne
         c += isfinite(a[i]) ? 0u : 1u;
     if (c) atomicAdd(bad, c);
 }
+#endif
 
 // ------------------------------------------------------------------ a1: voxelize
 
@@ -248,6 +252,7 @@ struct VoxArgs {
 // One thread per (slot, p): sums the coefficients of the probe's atoms in atom order
 // (deterministic), then multiplies by w_p.  Index math in FP64 with explicit IEEE
 // rounding (no FMA contraction) so that voxel indices equal the oracle's exactly.
+#ifndef DOCK_LAUNCHER_TU   // defined once, in dock.cu
 __global__ void k_voxelize(VoxArgs a)
 {
     int idx = blockIdx.x * blockDim.x + threadIdx.x;
@@ -303,8 +308,10 @@ __global__ void k_voxelize(VoxArgs a)
     const float wp = a.w[p];
     for (int v = 0; v < m3; v++) dst[v * RB] = dst[v * RB] * wp;
 }
+#endif
 
 // Lw [batch][P][m^3][RB]  ->  out [slot][P][m^3]   (debug export for dock_voxelize)
+#ifndef DOCK_LAUNCHER_TU   // defined once, in dock.cu
 __global__ void k_unpack_L(const float* __restrict__ Lw, float* __restrict__ out, int n_slots, int P, int m3)
 {
     int i = blockIdx.x * blockDim.x + threadIdx.x;
@@ -312,6 +319,7 @@ __global__ void k_unpack_L(const float* __restrict__ Lw, float* __restrict__ out
     int v = i % m3, p = (i / m3) % P, slot = i / (m3 * P);
     out[i] = Lw[((static_cast<size_t>(slot / RB) * P + p) * m3 + v) * RB + slot % RB];
 }
+#endif
 
 // ------------------------------------------------------------------ a2-a5: correlation
 
@@ -570,6 +578,7 @@ struct PoseOut {
 // equals the exact full-grid greedy when every warp list's 32nd key exceeds the last pick
 // (mu > key(c_k)); otherwise, or on candidate overflow, the rotation is flagged for the
 // exact fallback (DESIGN.md §Top-k exactness).
+#ifndef DOCK_LAUNCHER_TU   // defined once, in dock.cu
 __global__ void k_merge(MergeArgs a)
 {
     __shared__ unsigned long long picks_s[8][32];
@@ -622,6 +631,7 @@ __global__ void k_merge(MergeArgs a)
         a.fb_list[idx] = slot;
     }
 }
+#endif
 
 // ------------------------------------------------------------------ a6': exact greedy on a full grid
 
@@ -639,6 +649,7 @@ struct GreedyArgs {
 // spread over many CTAs per grid: every thread scans a strided share of the N^3 cells for
 // the best key that is farther than rho from picks 0..j-1, and the warp minima are combined
 // with one 64-bit atomicMin per warp into picks[g][j].
+#ifndef DOCK_LAUNCHER_TU   // defined once, in dock.cu
 __global__ void k_greedy_round(GreedyArgs a)
 {
     const int ctas_per_grid = gridDim.x / a.n;
@@ -662,8 +673,10 @@ __global__ void k_greedy_round(GreedyArgs a)
     best = warp_min_u64(best);
     if ((threadIdx.x & 31) == 0 && best != KEY_MAX) atomicMin(&pk[j], best);
 }
+#endif
 
 // Write the fallback poses (flag DOCK_POSE_FALLBACK) once all rounds are done.
+#ifndef DOCK_LAUNCHER_TU   // defined once, in dock.cu
 __global__ void k_greedy_emit(GreedyArgs a)
 {
     const int i = blockIdx.x * blockDim.x + threadIdx.x;
@@ -685,16 +698,20 @@ __global__ void k_greedy_emit(GreedyArgs a)
     }
     reinterpret_cast<PoseOut*>(a.poses)[static_cast<size_t>(slot) * a.k + j] = po;
 }
+#endif
 
+#ifndef DOCK_LAUNCHER_TU   // defined once, in dock.cu
 __global__ void k_fill_u64(unsigned long long* p, size_t n, unsigned long long v)
 {
     for (size_t i = blockIdx.x * static_cast<size_t>(blockDim.x) + threadIdx.x; i < n;
          i += static_cast<size_t>(gridDim.x) * blockDim.x)
         p[i] = v;
 }
+#endif
 
 // ------------------------------------------------------------------ per-call state reset
 
+#ifndef DOCK_LAUNCHER_TU   // defined once, in dock.cu
 __global__ void k_reset(unsigned long long* T, unsigned long long* mu, unsigned int* cnt, int n,
                         unsigned int* fb_cnt, unsigned int* cand_max)
 {
@@ -709,5 +726,6 @@ __global__ void k_reset(unsigned long long* T, unsigned long long* mu, unsigned 
         *cand_max = 0;
     }
 }
+#endif
 
 }  // namespace dk

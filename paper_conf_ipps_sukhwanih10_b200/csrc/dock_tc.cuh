@@ -13,8 +13,11 @@
 // K-major no-swizzle UMMA layout (core matrix = 8 rows x 16 B, rows 16 B apart, SBO = 128 B)
 // of "128 consecutive translations x (voxel vx, vx+1)" is the tile itself read at a start
 // address offset of the filter offset (vz, vy, vx); LBO = 16 B steps to voxel vx+1.
-// A (weights, K-major) streams through an 8-stage mbarrier ring (4 KB per K-step) and is
-// reused by the Q translation rows of a tile; D lives in TMEM (Q x 128 columns per buffer).
+// A (weights, K-major) streams through a <= 16-stage mbarrier ring (4 KB per K-step) and is
+// reused by the Q translation rows of a tile; D lives in TMEM (Q x NTT columns).
+// Two kernels: variant 1 (k_corr_tc: one channel group, both receptor boxes resident, NTT = 128) and
+// variant 2 (k_corr_tcs: any number of channel groups and m <= 8, receptor streamed z-plane by
+// z-plane through a ring, NTT in {64, 128, 160}).
 // Epilogue: one thread per (rotation, half of the rows) reads its TMEM lane with
 // tcgen05.ld and keeps an exact per-thread top-LIST key list (no score grid in HBM),
 // published at item end exactly like the FFMA engine (k_merge is shared).
@@ -38,16 +41,14 @@ constexpr int LIST = 16;        // per-thread candidate list (exact top-LIST key
 
 struct TcArgs {
     int nx, ny, nz;
-    int ntx, nty, ntz, ntiles;  // tiles: 128 x Q rows (y) x 1 (z)
+    int ntx, nty, ntz, ntiles;  // tiles: NTT x Q rows (y) x 1 (z)
     int G_ch;                   // channel groups of 4
     int n_slots, G, tiles_per_region;
-    int nsteps;                 // K-steps of A per tile (all passes, padded to multiples of KSTEPS)
-    int S1, S1p, S2, S2p;       // PAIR scheme: pass-1 steps (real, padded) and pass-2 steps (real, padded)
+    int nsteps;                 // K-steps of A per tile (all passes / units, padded to whole ring stages)
     const unsigned char* W;     // [block][step][WCHUNK]
-    int TXB, TYB, TZB;
-    int box_bytes;              // one channel group's receptor box
-    int rec_stage_bytes;        // G_ch * box_bytes rounded to 1024
-    int n_rec_stages;           // 1 or 2
+    int box_bytes;              // bytes of one receptor TMA box (variant 1: whole box; variant 2: one z-plane)
+    int rec_stage_bytes;        // variant 1: offset of the pair box; variant 2: one receptor ring slot (unit)
+    int n_rec_stages;           // variant 2: receptor ring depth (units)
     int wstages;                // weight ring depth (3..WSTAGES)
     int nepi;                   // epilogue warps (4, 8 or 16)
     // top-k
@@ -175,37 +176,134 @@ __device__ __forceinline__ void list_insert(unsigned long long (&L)[LIST], unsig
     L[0] = key < L[0] ? key : L[0];
 }
 
-__device__ __forceinline__ void cluster_sync_all()
+// ------------------------------------------------------------------ shared epilogue pieces
+
+// One 32-value chunk of scores (rotation of this thread, translations tbase + c0 + j, j < jmax valid)
+// into the per-thread exact top-LIST list; GRID writes the chunk to the score grid instead.
+template <bool GRID>
+__device__ __forceinline__ void epi_chunk(const uint32_t (&v)[32], unsigned long long (&lst)[LIST], float& th,
+                                          uint32_t& th_t, uint32_t tbase, int c0, int jmax, float* grid_row)
 {
-    asm volatile("barrier.cluster.arrive.release.aligned;\n\tbarrier.cluster.wait.acquire.aligned;" ::: "memory");
-}
-// Bulk copy global -> the same shared offset in every CTA of ctaMask, completing tx on each CTA's barrier.
-__device__ __forceinline__ void bulk_load_mc(void* dst, const void* src, unsigned bytes, uint64_t* bar, uint16_t mask)
-{
-    asm volatile(
-        "cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes.multicast::cluster [%0], [%1], %2, [%3], %4;" ::"r"(
-            dk::smem_u32(dst)),
-        "l"(src), "r"(bytes), "r"(dk::smem_u32(bar)), "h"(mask)
-        : "memory");
-}
-__device__ __forceinline__ void umma_commit_mc(uint64_t* bar, uint16_t mask)
-{
-    asm volatile(
-        "tcgen05.commit.cta_group::1.mbarrier::arrive::one.shared::cluster.multicast::cluster.b64 [%0], %1;" ::"r"(
-            dk::smem_u32(bar)),
-        "h"(mask)
-        : "memory");
+    if constexpr (GRID) {
+#pragma unroll
+        for (int j = 0; j < 32; j++)
+            if (j < jmax) grid_row[c0 + j] = __uint_as_float(v[j]);
+    } else {
+        // fast check: one FMNMX per value; the insertion path is rare after warm-up
+        float mn = __uint_as_float(v[0]);
+#pragma unroll
+        for (int j = 1; j < 32; j++) mn = fminf(mn, __uint_as_float(v[j]));
+        // exact gate: a strictly better score, or a tie that could carry a smaller t_lin (exact-zero
+        // scores in empty space tie constantly)
+        if (mn < th || (mn == th && tbase + c0 < th_t)) {
+            // rare path: bitmask of candidates, each extracted with a 5-level select tree (no local memory)
+            uint32_t msk = 0;
+#pragma unroll
+            for (int j = 0; j < 32; j++) msk |= (__uint_as_float(v[j]) <= th && j < jmax) ? (1u << j) : 0u;
+            while (msk) {
+                const int j = __ffs(msk) - 1;
+                msk &= msk - 1;
+                const float sv = __uint_as_float(select32(v, j));
+                if (sv <= th) {
+                    const unsigned long long key = dk::make_key(sv, tbase + c0 + j);
+                    if (key < lst[LIST - 1]) {
+                        list_insert(lst, key);
+                        th = dk::key_score_bound(static_cast<uint32_t>(lst[LIST - 1] >> 32));
+                        th_t = static_cast<uint32_t>(lst[LIST - 1] & 0xffffffffu);
+                    }
+                }
+            }
+        }
+    }
 }
 
-// Shared-memory box geometry of the PAIR scheme (must match make_tc_plan): x extent, y extent.
-__host__ __device__ constexpr int pair_txb(int m)
+// Item end: bound T_w from k list entries pairwise farther than 2*rho apart, then
+// publish bound, mu and the keys <= T (k_merge finishes the greedy).  Loops over the register list
+// are fully unrolled (static indices keep it in registers).
+__device__ __forceinline__ void epi_publish(const unsigned long long (&lst)[LIST], int slot, const TcArgs& a)
 {
-    return (128 + (m + 1) / 2 * 2 - 1) > (4 * ((m + 3) / 4) + 126) ? (128 + (m + 1) / 2 * 2 - 1)
-                                                                     : (4 * ((m + 3) / 4) + 126);
+    unsigned long long Tw = KEY_MAX;
+    uint32_t chosen[32];
+    int nc = 0;
+#pragma unroll
+    for (int i = 0; i < LIST; i++) {
+        const unsigned long long key = lst[i];
+        if (key != KEY_MAX && nc < a.k) {
+            const uint32_t t = static_cast<uint32_t>(key & 0xffffffffu);
+            bool far = true;
+            for (int c = 0; c < nc; c++) far = far && dk::cheb_cyc(t, chosen[c], a.nx, a.ny, a.nz) > 2 * a.rho;
+            if (far) {
+                chosen[nc] = t;
+                nc++;
+                if (nc == a.k) Tw = key;
+            }
+        }
+    }
+    const unsigned long long old = atomicMin(&a.T[slot], Tw);
+    const unsigned long long Tn = old < Tw ? old : Tw;
+    atomicMin(&a.mu[slot], lst[LIST - 1]);
+#pragma unroll
+    for (int i = 0; i < LIST; i++) {
+        const unsigned long long key = lst[i];
+        if (key != KEY_MAX && key <= Tn) {
+            const unsigned pos = atomicAdd(&a.cnt[slot], 1u);
+            if (pos < static_cast<unsigned>(a.cap)) a.cand[static_cast<size_t>(slot) * a.cap + pos] = key;
+        }
+    }
+}
+
+// Epilogue of one tile: Q accumulator rows of NTT translations, TMEM columns [q * NTT, (q + 1) * NTT).
+// Warp (quarter, class cls) reads the TMEM lanes of its quarter (lane = rotation); rows are drained in
+// order q = 0..Q-1 and each row is released (tm_empty[q]) as soon as the warp's last chunk of it is in
+// registers, before that chunk is processed.  Within row q the warp takes the 32-column chunks
+// jj = cls, cls + nclass, ... at column ((q + jj) mod NCH) * 32 ("diagonal" classes: over the rows of a
+// tile a class's cells are spread like a row class).
+template <int NTT, int Q, bool GRID>
+__device__ __forceinline__ void epi_tile(const TcArgs& a, uint32_t tmem, uint64_t* tm_empty, int quarter, int cls,
+                                         int nclass, int lane, int slot, bool rot_ok, int tx, int ty, int tz,
+                                         unsigned long long (&lst)[LIST], float& th, uint32_t& th_t, bool tr,
+                                         long long& tw1)
+{
+    constexpr int NCH = NTT / 32;
+    const int x0 = tx * NTT;
+    for (int q = 0; q < Q; q++) {
+        const int y = ty * Q + q, z = tz;
+        const bool row_ok = rot_ok && y < a.ny && z < a.nz;
+        const uint32_t tbase = static_cast<uint32_t>((z * a.ny + y) * a.nx + x0);
+        if (a.dbg == 1 || cls >= NCH) {   // diagnostic (no TMEM drain), or no chunk of this row for this class
+            __syncwarp();
+            if (lane == 0) dk::mbar_arrive(&tm_empty[q]);
+            continue;
+        }
+#pragma unroll 1
+        for (int jj = cls; jj < NCH; jj += nclass) {
+            const int c0 = ((q + jj) % NCH) * 32;
+            uint32_t v[32];
+            const long long tl0 = tr ? clock64() : 0;
+            tmem_ld32(tmem + (static_cast<uint32_t>(quarter * 32) << 16) + q * NTT + c0, v);
+            if (tr) tw1 += clock64() - tl0;
+            if (jj + nclass >= NCH) {   // the warp's last chunk of this row is in registers: release the row
+                tc_fence_before();
+                __syncwarp();
+                if (lane == 0) dk::mbar_arrive(&tm_empty[q]);
+            }
+            if (!row_ok || a.dbg == 2) continue;
+            epi_chunk<GRID>(v, lst, th, th_t, tbase, c0, min(32, a.nx - x0 - c0),
+                            GRID ? a.grid + static_cast<size_t>(slot) * a.nx * a.ny * a.nz + tbase : nullptr);
+        }
+    }
+}
+
+// Shared-memory box geometry of the PAIR scheme (must match make_tc_plan): x extent of the (hi,lo) box
+// and of the (hi(x),hi(x+1)) box for NTT translations per row.
+__host__ __device__ constexpr int pair_txb(int m, int ntt = NT)
+{
+    return (ntt + (m + 1) / 2 * 2 - 1) > (4 * ((m + 3) / 4) + ntt - 2) ? (ntt + (m + 1) / 2 * 2 - 1)
+                                                                       : (4 * ((m + 3) / 4) + ntt - 2);
 }
 // Byte offset of K-step s inside the PAIR pass-1 box ((hi,lo) voxels, 2 per K-step) and pass-2 box
 // ((hi(x),hi(x+1)) slots, 4 voxels per K-step); padding steps (zero weights) re-read the last real
-// step's voxels (a plane still resident in the z-plane pipeline of dock_tc_skew.cuh).
+// step's voxels.
 __host__ __device__ constexpr uint32_t pair_off1(int m, int s, uint32_t row16, uint32_t rowTY)
 {
     const int mxp = (m + 1) / 2, t = s < m * m * mxp ? s : m * m * mxp - 1;
@@ -219,39 +317,45 @@ __host__ __device__ constexpr uint32_t pair_off2(int m, int s, uint32_t row16, u
            static_cast<uint32_t>(t % mxq) * 64u;
 }
 
-// CL = 1: one CTA per item.  CL = 2: a cluster of two CTAs works on the same rotation block
-// (two regions with the same number of tiles); each CTA's producer fetches half of every
-// weight chunk and multicasts it into both CTAs' rings, and each MMA warp releases a ring
-// slot in both CTAs -- the weight stream from L2 is halved, which lets Q = 2 rows per TMEM
-// buffer with NBUF = 2 buffers (epilogue overlapped with the next tile's MMAs).
-// PAIR (one channel group): pass 1 reads the (hi, lo) receptor box -> Rhi*Whi + Rlo*Whi over 2 voxels
-// per MMA; pass 2 reads a second box whose 16-B slot x holds (Rhi(x), Rhi(x+1)), so one K = 16 MMA
-// covers 4 voxels of Rhi*Wlo (chunk LBO = 32 B): 3 MMAs per 4 voxels instead of 4.
-template <int M, int Q, int NBUF, int CL, bool PAIR, bool GRID>
+// ------------------------------------------------------------------ variant 1: resident receptor boxes
+//
+// One channel group (P <= 4), PAIR scheme: pass 1 reads the (hi, lo) receptor box -> Rhi*Whi + Rlo*Whi
+// over 2 voxels per MMA; pass 2 reads a second box whose 16-B slot x holds (Rhi(x), Rhi(x+1)), so one
+// K = 16 MMA covers 4 voxels of Rhi*Wlo (chunk LBO = 32 B): 3 MMAs per 4 voxels instead of 4.  Both
+// whole boxes (all m z-planes, Q = 4 rows + halo) are resident; the main box is released after pass 1
+// and the pair box after pass 2, so one buffer of each gives full TMA/MMA overlap.  One TMEM buffer of
+// Q x 128 columns; rows are released one by one by the epilogue and restarted in that order.
+template <int M, bool GRID>
 __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__ CUtensorMap tmap,
                                                           const __grid_constant__ CUtensorMap tmap_pair, const TcArgs a)
 {
+    constexpr int Q = 4;
     constexpr int KS = KSTEPS;                 // K-steps per weight-ring stage (one wait/commit per KS steps)
     constexpr unsigned STAGE = KS * WCHUNK;
-    static_assert(Q * NBUF * NT <= 512, "TMEM has 512 columns");
-    constexpr int MXP = (M + 1) / 2;   // voxel pairs along x (K = 16 = 2 voxels x 8 channels)
+    constexpr int MXP = (M + 1) / 2, MXQ = (M + 3) / 4;
+    constexpr int S1 = M * M * MXP, S1P = (S1 + KS - 1) / KS * KS;
+    constexpr int S2 = M * M * MXQ, S2P = (S2 + KS - 1) / KS * KS;
+    constexpr int NSTEPS = S1P + S2P;
+    constexpr uint32_t ROW16 = static_cast<uint32_t>(pair_txb(M)) * 16u;
+    constexpr uint32_t ROWTY = static_cast<uint32_t>(Q + M - 1) * ROW16;
+    static_assert(Q * NT <= 512, "TMEM has 512 columns");
     extern __shared__ __align__(1024) unsigned char smem[];
-    __shared__ uint64_t bars[2 * 2 + 2 * WSTAGES + NBUF + NBUF * Q];
+    __shared__ uint64_t bars[2 * 2 + 2 * WSTAGES + 1 + Q];
     __shared__ uint32_t tmem_base_s;
     uint64_t* rec_full = bars;
     uint64_t* rec_empty = bars + 2;
     uint64_t* w_full = bars + 4;
     uint64_t* w_empty = w_full + WSTAGES;
     uint64_t* tm_full = w_empty + WSTAGES;
-    uint64_t* tm_empty = tm_full + NBUF;   // [NBUF][Q]: per accumulator row, so the next tile restarts row by row
+    uint64_t* tm_empty = tm_full + 1;   // [Q]: per accumulator row, so the next tile restarts row by row
 
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     const int block = blockIdx.x / a.G, region = blockIdx.x % a.G;
     const int tile_begin = region * a.tiles_per_region;
     const int tile_end = min(a.ntiles, tile_begin + a.tiles_per_region);
     const int n_tiles = tile_end - tile_begin;
-    unsigned char* rec_smem = smem;
-    unsigned char* w_smem = smem + a.n_rec_stages * a.rec_stage_bytes;
+    unsigned char* rec_smem = smem;   // [main box | pair box], a.rec_stage_bytes each
+    unsigned char* w_smem = smem + 2 * a.rec_stage_bytes;
 
     if (threadIdx.x == 0) {
         for (int i = 0; i < 2; i++) {
@@ -260,10 +364,10 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
         }
         for (int i = 0; i < a.wstages; i++) {
             dk::mbar_init(&w_full[i], 1);
-            dk::mbar_init(&w_empty[i], CL);
+            dk::mbar_init(&w_empty[i], 1);
         }
-        for (int i = 0; i < NBUF; i++) dk::mbar_init(&tm_full[i], 1);
-        for (int i = 0; i < NBUF * Q; i++) dk::mbar_init(&tm_empty[i], a.nepi);
+        dk::mbar_init(&tm_full[0], 1);
+        for (int i = 0; i < Q; i++) dk::mbar_init(&tm_empty[i], a.nepi);
         dk::fence_mbar_init();
     }
     if (warp == 1) {
@@ -273,12 +377,8 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
     }
     tc_fence_before();
     __syncthreads();
-    if constexpr (CL > 1) cluster_sync_all();   // peers' barriers are initialised before any multicast
     tc_fence_after();
     const uint32_t tmem = tmem_base_s;
-    uint32_t crank = 0;
-    if constexpr (CL > 1) asm volatile("mov.u32 %0, %%cluster_ctarank;" : "=r"(crank));
-    constexpr uint16_t CMASK = (1u << CL) - 1u;
 
     const bool tr = a.trace != nullptr;
     long long tw0 = 0, tw1 = 0, tw2 = 0, tstart = tr ? clock64() : 0;   // per-role trace accumulators
@@ -287,111 +387,64 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
             // ------------------------------------------------ TMA producer (warp-converged, one elected lane)
             if (elect_one()) {
                 dk::prefetch_tmap(&tmap);
-                if constexpr (PAIR) dk::prefetch_tmap(&tmap_pair);
+                dk::prefetch_tmap(&tmap_pair);
             }
-            const unsigned char* wsrc = a.W + static_cast<size_t>(block) * a.nsteps * WCHUNK;
+            const unsigned char* wsrc = a.W + static_cast<size_t>(block) * NSTEPS * WCHUNK;
             int ws = 0, wph = 0;                  // weight ring slot / phase
             int wuse = 0;
-            auto stream_weights = [&](int s0, int s1) {
-                for (int s = s0; s < s1; s += KS) {
-                    if (wuse >= a.wstages) twait(&w_empty[ws], wph ^ 1, tr, tw0);
-                    if (elect_one()) {
-                        dk::mbar_arrive_expect_tx(&w_full[ws], STAGE);
-                        if constexpr (CL == 1) {
-                            dk::bulk_load(w_smem + static_cast<size_t>(ws) * STAGE,
-                                          wsrc + static_cast<size_t>(s) * WCHUNK, STAGE, &w_full[ws]);
-                        } else {
-                            constexpr unsigned HALF = STAGE / CL;
-                            bulk_load_mc(w_smem + static_cast<size_t>(ws) * STAGE + crank * HALF,
-                                         wsrc + static_cast<size_t>(s) * WCHUNK + crank * HALF, HALF, &w_full[ws],
-                                         CMASK);
-                        }
-                    }
-                    __syncwarp();
-                    wuse++;
-                    if (++ws == a.wstages) {
-                        ws = 0;
-                        wph ^= 1;
-                    }
-                }
-            };
-            if constexpr (PAIR) {
-                // Receptor boxes are issued as soon as their buffer frees: the producer polls the
-                // release barriers between weight stages (main(t+1) needs pass 1 of t done, pair(t+1)
-                // pass 2 of t), and blocks only right before the first stage that needs a box.
-                int pm = 0, pp = 0;   // next main / pair box (tile index) to load
-                auto issue_box = [&](int which, int t) {
-                    const int tile = tile_begin + t;
-                    const int tx = tile % a.ntx, ty = (tile / a.ntx) % a.nty, tz = tile / (a.ntx * a.nty);
-                    if (elect_one()) {
-                        dk::mbar_arrive_expect_tx(&rec_full[which], a.box_bytes);
-                        tma_load_5d(rec_smem + which * a.rec_stage_bytes, which ? &tmap_pair : &tmap, 0, tx * NT,
-                                    ty * Q, tz, 0, &rec_full[which]);
-                    }
-                    __syncwarp();
-                };
-                auto poll = [&](int ti) {
-                    if (pm < n_tiles && pm <= ti + 1 && (pm == 0 || dk::mbar_test(&rec_empty[0], (pm - 1) & 1)))
-                        issue_box(0, pm++);
-                    if (pp < n_tiles && pp <= ti + 1 && (pp == 0 || dk::mbar_test(&rec_empty[1], (pp - 1) & 1)))
-                        issue_box(1, pp++);
-                };
-                auto ensure = [&](int which, int t) {
-                    int& nx = which ? pp : pm;
-                    if (nx == t) {
-                        if (t > 0) twait(&rec_empty[which], (t - 1) & 1, tr, tw1);
-                        issue_box(which, nx++);
-                    }
-                };
-                for (int ti = 0; ti < n_tiles; ti++) {
-                    ensure(0, ti);
-                    for (int s = 0; s < a.S1p; s += KS) {
-                        poll(ti);
-                        stream_weights(s, s + KS);
-                    }
-                    ensure(1, ti);
-                    for (int s = a.S1p; s < a.nsteps; s += KS) {
-                        poll(ti);
-                        stream_weights(s, s + KS);
-                    }
-                }
-            } else {
-            for (int ti = 0; ti < n_tiles; ti++) {
-                const int tile = tile_begin + ti;
-                const int rs = ti % a.n_rec_stages, ruse = ti / a.n_rec_stages;
-                if (ruse > 0) twait(&rec_empty[rs], (ruse - 1) & 1, tr, tw1);
-                const int tx = tile % a.ntx, ty = (tile / a.ntx) % a.nty, tz = tile / (a.ntx * a.nty);
-                unsigned char* rdst = rec_smem + static_cast<size_t>(rs) * a.rec_stage_bytes;
+            auto stream_weights = [&](int s) {
+                if (wuse >= a.wstages) twait(&w_empty[ws], wph ^ 1, tr, tw0);
                 if (elect_one()) {
-                    dk::mbar_arrive_expect_tx(&rec_full[rs], a.G_ch * a.box_bytes);
-                    for (int g = 0; g < a.G_ch; g++)
-                        tma_load_5d(rdst + static_cast<size_t>(g) * a.box_bytes, &tmap, 0, tx * NT, ty * Q, tz, g,
-                                    &rec_full[rs]);
+                    dk::mbar_arrive_expect_tx(&w_full[ws], STAGE);
+                    dk::bulk_load(w_smem + static_cast<size_t>(ws) * STAGE, wsrc + static_cast<size_t>(s) * WCHUNK,
+                                  STAGE, &w_full[ws]);
                 }
                 __syncwarp();
-                for (int s = 0; s < a.nsteps; s += KS) {
-                    if (wuse >= a.wstages) twait(&w_empty[ws], wph ^ 1, tr, tw0);
-                    if (elect_one()) {
-                        dk::mbar_arrive_expect_tx(&w_full[ws], STAGE);
-                        if constexpr (CL == 1) {
-                            dk::bulk_load(w_smem + static_cast<size_t>(ws) * STAGE,
-                                          wsrc + static_cast<size_t>(s) * WCHUNK, STAGE, &w_full[ws]);
-                        } else {
-                            constexpr unsigned HALF = STAGE / CL;
-                            bulk_load_mc(w_smem + static_cast<size_t>(ws) * STAGE + crank * HALF,
-                                         wsrc + static_cast<size_t>(s) * WCHUNK + crank * HALF, HALF, &w_full[ws],
-                                         CMASK);
-                        }
-                    }
-                    __syncwarp();
-                    wuse++;
-                    if (++ws == a.wstages) {
-                        ws = 0;
-                        wph ^= 1;
-                    }
+                wuse++;
+                if (++ws == a.wstages) {
+                    ws = 0;
+                    wph ^= 1;
+                }
+            };
+            // Receptor boxes are issued as soon as their buffer frees: the producer polls the release
+            // barriers between weight stages (main(t+1) needs pass 1 of t done, pair(t+1) pass 2 of t),
+            // and blocks only right before the first stage that needs a box.
+            int pm = 0, pp = 0;   // next main / pair box (tile index) to load
+            auto issue_box = [&](int which, int t) {
+                const int tile = tile_begin + t;
+                const int tx = tile % a.ntx, ty = (tile / a.ntx) % a.nty, tz = tile / (a.ntx * a.nty);
+                if (elect_one()) {
+                    dk::mbar_arrive_expect_tx(&rec_full[which], a.box_bytes);
+                    tma_load_5d(rec_smem + which * a.rec_stage_bytes, which ? &tmap_pair : &tmap, 0, tx * NT, ty * Q,
+                                tz, 0, &rec_full[which]);
+                }
+                __syncwarp();
+            };
+            auto poll = [&](int ti) {
+                if (pm < n_tiles && pm <= ti + 1 && (pm == 0 || dk::mbar_test(&rec_empty[0], (pm - 1) & 1)))
+                    issue_box(0, pm++);
+                if (pp < n_tiles && pp <= ti + 1 && (pp == 0 || dk::mbar_test(&rec_empty[1], (pp - 1) & 1)))
+                    issue_box(1, pp++);
+            };
+            auto ensure = [&](int which, int t) {
+                int& nx = which ? pp : pm;
+                if (nx == t) {
+                    if (t > 0) twait(&rec_empty[which], (t - 1) & 1, tr, tw1);
+                    issue_box(which, nx++);
+                }
+            };
+            for (int ti = 0; ti < n_tiles; ti++) {
+                ensure(0, ti);
+                for (int s = 0; s < S1P; s += KS) {
+                    poll(ti);
+                    stream_weights(s);
+                }
+                ensure(1, ti);
+                for (int s = S1P; s < NSTEPS; s += KS) {
+                    poll(ti);
+                    stream_weights(s);
                 }
             }
-            }   // !PAIR
             if (tr && elect_one()) {
                 atomicAdd(&a.trace[TR_PROD_TOTAL], static_cast<unsigned long long>(clock64() - tstart));
                 atomicAdd(&a.trace[TR_PROD_WEMPTY], static_cast<unsigned long long>(tw0));
@@ -400,41 +453,20 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                 atomicAdd(&a.trace[TR_TILES], static_cast<unsigned long long>(n_tiles));
             }
             __syncwarp();
-            if constexpr (CL > 1) {
-                // drain: every ring slot's last release (from both MMA warps) has arrived before exit
-                for (int i = 0; i < min(wuse, a.wstages); i++) {
-                    dk::mbar_wait(&w_empty[ws], wph ^ 1);
-                    if (++ws == a.wstages) {
-                        ws = 0;
-                        wph ^= 1;
-                    }
-                }
-            }
         } else if (warp == 1) {
-            // ------------------------------------------------ MMA issuer (warp-converged, one elected lane)
-            // One elected block per ring stage (KS K-steps x Q rows = KS*Q MMAs): the warp re-converges
-            // once per stage, not once per K-step (the re-convergence waits for the tcgen05 issue).
+            // ------------------------------------------------ MMA issuer (one thread runs the whole schedule)
+            // The stage loops are unrolled so every descriptor offset is an immediate and the tcgen05 queue
+            // stays fed (issuing per K-step from a converged warp capped the tensor pipe at 40-47 %).
             constexpr uint32_t idesc = umma_idesc(ROT, NT);
-            constexpr int MXQ = (M + 3) / 4;   // PAIR pass 2: 4-voxel groups along x
             const uint32_t rec0 = dk::smem_u32(rec_smem), w0 = dk::smem_u32(w_smem);
-            const uint64_t dA0 = umma_desc(w0, ROT * 16, 128);                      // + (slot offset >> 4)
-            const uint64_t dB0 = umma_desc(rec0, 16, 128);                          // + (voxel offset >> 4)
-            const uint64_t dP0 = umma_desc(rec0 + (PAIR ? a.rec_stage_bytes : 0), 32, 128);
-            const uint32_t row16 = static_cast<uint32_t>(a.TXB) * 16u;
-            const uint32_t rowTY = static_cast<uint32_t>(a.TYB) * row16;
-            if constexpr (PAIR && CL == 1) {
-            // Lean issue loop: one thread runs the whole schedule (no per-stage warp re-convergence), the
-            // stage loops are unrolled so every descriptor offset is an immediate; the tcgen05 queue stays fed.
-            constexpr int S1 = M * M * MXP, S1P = (S1 + KS - 1) / KS * KS;
-            constexpr int S2 = M * M * MXQ, S2P = (S2 + KS - 1) / KS * KS;
-            constexpr uint32_t ROW16 = static_cast<uint32_t>(pair_txb(M)) * 16u;
-            constexpr uint32_t ROWTY = static_cast<uint32_t>(Q + M - 1) * ROW16;
+            const uint64_t dA0 = umma_desc(w0, ROT * 16, 128);                 // + (slot offset >> 4)
+            const uint64_t dB0 = umma_desc(rec0, 16, 128);                     // + (voxel offset >> 4)
+            const uint64_t dP0 = umma_desc(rec0 + a.rec_stage_bytes, 32, 128);
             if (elect_one()) {
                 uint32_t ws = 0, wph = 0;
                 const uint32_t nws = static_cast<uint32_t>(a.wstages);
                 for (int ti = 0; ti < n_tiles; ti++) {
-                    const int buf = ti % NBUF, buse = ti / NBUF;
-                    const uint32_t dcol = tmem + static_cast<uint32_t>(buf * Q * NT);
+                    const uint32_t dcol = tmem;
                     twait(&rec_full[0], ti & 1, tr, tw2);
                     tc_fence_after();
 #pragma unroll
@@ -442,11 +474,11 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                         twait(&w_full[ws], wph, tr, tw1);
                         tc_fence_after();
                         const uint64_t da0 = dA0 + ((ws * STAGE) >> 4);
-                        if (st == 0 && buse > 0) {
+                        if (st == 0 && ti > 0) {
                             // accumulator rows are released one by one while the epilogue drains them
 #pragma unroll
                             for (int q = 0; q < Q; q++) {
-                                twait(&tm_empty[buf * Q + q], (buse - 1) & 1, tr, tw0);
+                                twait(&tm_empty[q], (ti - 1) & 1, tr, tw0);
                                 tc_fence_after();
 #pragma unroll
                                 for (int ks = 0; ks < KS; ks++)
@@ -491,7 +523,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                         }
                     }
                     umma_commit(&rec_empty[1]);
-                    umma_commit(&tm_full[buf]);
+                    umma_commit(&tm_full[0]);
                 }
                 if (tr) {
                     atomicAdd(&a.trace[TR_MMA_TOTAL], static_cast<unsigned long long>(clock64() - tstart));
@@ -501,118 +533,11 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                 }
             }
             __syncwarp();
-            } else {
-            int ws = 0, wph = 0;
-            // B descriptor of K-step s: PAIR pass 1 (kind 0), PAIR pass 2 (kind 1) or the 2-pass scheme (kind 2)
-            auto bdesc = [&](int kind, int s, uint32_t rofs) -> uint64_t {
-                if (kind == 0) {
-                    if (s >= a.S1) return dB0;
-                    const int vxp = s % MXP, vy = (s / MXP) % M, vz = s / (MXP * M);
-                    return dB0 + ((rofs + vz * rowTY + vy * row16 + vxp * 32u) >> 4);
-                }
-                if (kind == 1) {
-                    if (s >= a.S2) return dP0;
-                    const int vxq = s % MXQ, vy = (s / MXQ) % M, vz = s / (MXQ * M);
-                    return dP0 + ((vz * rowTY + vy * row16 + vxq * 64u) >> 4);
-                }
-                const int vxp = s % MXP, vy = (s / MXP) % M, vz = (s / (MXP * M)) % M;
-                const int g = s / (MXP * M * M * 2);
-                return dB0 + ((rofs + g * a.box_bytes + vz * rowTY + vy * row16 + vxp * 32u) >> 4);
-            };
-            // rel != nullptr: first stage of a tile whose accumulator rows are still being drained --
-            // issue row-major, each row right after the epilogue released it (rel[q], parity relph)
-            auto issue_stage = [&](int kind, int s0, uint32_t rofs, uint32_t dcol, bool first, uint64_t* rel,
-                                   int relph) {
-                twait(&w_full[ws], wph, tr, tw1);
-                tc_fence_after();
-                const uint64_t da0 = dA0 + ((static_cast<uint32_t>(ws) * STAGE) >> 4);
-                if (rel) {
-#pragma unroll
-                    for (int q = 0; q < Q; q++) {
-                        twait(&rel[q], relph, tr, tw0);
-                        tc_fence_after();
-                        if (elect_one()) {
-#pragma unroll
-                            for (int ks = 0; ks < KS; ks++)
-                                umma_bf16(dcol + q * NT, da0 + ((ks * WCHUNK) >> 4),
-                                          bdesc(kind, s0 + ks, rofs) + ((q * row16) >> 4), idesc, ks == 0 ? 0u : 1u);
-                        }
-                        __syncwarp();
-                    }
-                } else if (elect_one()) {
-#pragma unroll
-                    for (int ks = 0; ks < KS; ks++) {
-                        const uint64_t db = bdesc(kind, s0 + ks, rofs);
-                        const uint64_t da = da0 + ((ks * WCHUNK) >> 4);
-#pragma unroll
-                        for (int q = 0; q < Q; q++)
-                            umma_bf16(dcol + q * NT, da, db + ((q * row16) >> 4), idesc, (first && ks == 0) ? 0u : 1u);
-                    }
-                }
-                __syncwarp();
-                if (elect_one()) {
-                    if constexpr (CL == 1) umma_commit(&w_empty[ws]);
-                    else umma_commit_mc(&w_empty[ws], CMASK);
-                }
-                __syncwarp();
-                if (++ws == a.wstages) {
-                    ws = 0;
-                    wph ^= 1;
-                }
-            };
-            for (int ti = 0; ti < n_tiles; ti++) {
-                const int buf = ti % NBUF, buse = ti / NBUF;
-                const uint32_t dcol = tmem + static_cast<uint32_t>(buf * Q * NT);
-                if constexpr (PAIR) {
-                    twait(&rec_full[0], ti & 1, tr, tw2);
-                    tc_fence_after();
-                    uint64_t* rel = buse > 0 ? &tm_empty[buf * Q] : nullptr;
-                    for (int s = 0; s < a.S1p; s += KS)
-                        issue_stage(0, s, 0u, dcol, s == 0, s == 0 ? rel : nullptr, (buse - 1) & 1);
-                    if (elect_one()) umma_commit(&rec_empty[0]);
-                    __syncwarp();
-                    twait(&rec_full[1], ti & 1, tr, tw2);
-                    tc_fence_after();
-                    for (int s = 0; s < a.S2p; s += KS) issue_stage(1, s, 0u, dcol, false, nullptr, 0);
-                    if (elect_one()) {
-                        umma_commit(&rec_empty[1]);
-                        umma_commit(&tm_full[buf]);
-                    }
-                    __syncwarp();
-                } else {
-                    const int rs = ti % a.n_rec_stages, ruse = ti / a.n_rec_stages;
-                    twait(&rec_full[rs], ruse & 1, tr, tw2);
-                    tc_fence_after();
-                    const uint32_t rofs = static_cast<uint32_t>(rs * a.rec_stage_bytes);
-                    uint64_t* rel = buse > 0 ? &tm_empty[buf * Q] : nullptr;
-                    for (int s = 0; s < a.nsteps; s += KS)
-                        issue_stage(2, s, rofs, dcol, s == 0, s == 0 ? rel : nullptr, (buse - 1) & 1);
-                    if (elect_one()) {
-                        umma_commit(&tm_full[buf]);
-                        umma_commit(&rec_empty[rs]);
-                    }
-                    __syncwarp();
-                }
-            }
-            if (tr && elect_one()) {
-                atomicAdd(&a.trace[TR_MMA_TOTAL], static_cast<unsigned long long>(clock64() - tstart));
-                atomicAdd(&a.trace[TR_MMA_TMEMPTY], static_cast<unsigned long long>(tw0));
-                atomicAdd(&a.trace[TR_MMA_WFULL], static_cast<unsigned long long>(tw1));
-                atomicAdd(&a.trace[TR_MMA_RFULL], static_cast<unsigned long long>(tw2));
-            }
-            __syncwarp();
-            }   // generic issue loop
         } else {
             // ------------------------------------------------ epilogue warps
-            // Warp (quarter, class cls) reads TMEM lanes of its quarter (lane = rotation).  Rows are
-            // drained in order q = 0..Q-1 so each accumulator row is released (tm_empty[buf][q]) as soon as
-            // its last chunk is in registers, before the chunk is processed; within row q the warp takes the
-            // 32-column chunks c = (q + cls + j * nclass) mod 4 ("diagonal" classes: over the Q rows of a
-            // tile a class covers one chunk per row, so the cells of a list are spread like a row class).
             const int quarter = warp & 3;
             const int cls = (warp - 2) >> 2;
             const int nclass = a.nepi >> 2;
-            constexpr int NCH = NT / 32;                         // 32-column chunks per row
             const int r = quarter * 32 + lane;                  // rotation within the block (TMEM lane)
             const int slot = block * ROT + r;
             const bool rot_ok = slot < a.n_slots;
@@ -623,68 +548,10 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
             uint32_t th_t = 0xffffffffu;             // t_lin of the list's last key
             int tx = tile_begin % a.ntx, ty = (tile_begin / a.ntx) % a.nty, tz = tile_begin / (a.ntx * a.nty);
             for (int ti = 0; ti < n_tiles; ti++) {
-                const int buf = ti % NBUF, buse = ti / NBUF;
-                twait(&tm_full[buf], buse & 1, tr, tw0);
+                twait(&tm_full[0], ti & 1, tr, tw0);
                 tc_fence_after();
-                if (a.dbg == 1) {   // diagnostic: no TMEM drain
-                    __syncwarp();
-                    if (lane == 0)
-                        for (int q = 0; q < Q; q++) dk::mbar_arrive(&tm_empty[buf * Q + q]);
-                } else {
-                    const int x0 = tx * NT;
-                    for (int q = 0; q < Q; q++) {
-                        const int y = ty * Q + q, z = tz;
-                        const bool row_ok = rot_ok && y < a.ny && z < a.nz;
-                        const uint32_t tbase = static_cast<uint32_t>((z * a.ny + y) * a.nx + x0);
-#pragma unroll 1
-                        for (int j = 0; j < NCH / nclass; j++) {
-                            const int c0 = ((q + cls + j * nclass) & (NCH - 1)) * 32;
-                            uint32_t v[32];
-                            const long long tl0 = tr ? clock64() : 0;
-                            tmem_ld32(tmem + (static_cast<uint32_t>(quarter * 32) << 16) + (buf * Q + q) * NT + c0, v);
-                            if (tr) tw1 += clock64() - tl0;
-                            if (j == NCH / nclass - 1) {   // the row's last chunk is in registers: release the row
-                                tc_fence_before();
-                                __syncwarp();
-                                if (lane == 0) dk::mbar_arrive(&tm_empty[buf * Q + q]);
-                            }
-                            if (!row_ok || a.dbg == 2) continue;
-                            if constexpr (GRID) {
-                                float* out = a.grid + static_cast<size_t>(slot) * a.nx * a.ny * a.nz + tbase;
-#pragma unroll
-                                for (int jj = 0; jj < 32; jj++)
-                                    if (x0 + c0 + jj < a.nx) out[c0 + jj] = __uint_as_float(v[jj]);
-                            } else {
-                                // fast check: one FMNMX per value; the insertion path is rare after warm-up
-                                float mn = __uint_as_float(v[0]);
-#pragma unroll
-                                for (int jj = 1; jj < 32; jj++) mn = fminf(mn, __uint_as_float(v[jj]));
-                                // exact gate: a strictly better score, or a tie that could carry a smaller t_lin
-                                if (mn < th || (mn == th && tbase + c0 < th_t)) {
-                                    // rare path: bitmask of candidates, each extracted with a 5-level select tree
-                                    const int jmax = min(32, a.nx - x0 - c0);
-                                    uint32_t msk = 0;
-#pragma unroll
-                                    for (int jj = 0; jj < 32; jj++)
-                                        msk |= (__uint_as_float(v[jj]) <= th && jj < jmax) ? (1u << jj) : 0u;
-                                    while (msk) {
-                                        const int jj = __ffs(msk) - 1;
-                                        msk &= msk - 1;
-                                        const float sv = __uint_as_float(select32(v, jj));
-                                        if (sv <= th) {
-                                            const unsigned long long key = dk::make_key(sv, tbase + c0 + jj);
-                                            if (key < lst[LIST - 1]) {
-                                                list_insert(lst, key);
-                                                th = dk::key_score_bound(static_cast<uint32_t>(lst[LIST - 1] >> 32));
-                                                th_t = static_cast<uint32_t>(lst[LIST - 1] & 0xffffffffu);
-                                            }
-                                        }
-                                    }
-                                }
-                            }
-                        }
-                    }
-                }
+                epi_tile<NT, Q, GRID>(a, tmem, tm_empty, quarter, cls, nclass, lane, slot, rot_ok, tx, ty, tz, lst, th,
+                                      th_t, tr, tw1);
                 if (++tx == a.ntx) {
                     tx = 0;
                     if (++ty == a.nty) {
@@ -700,51 +567,277 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                 atomicAdd(&a.trace[TR_EPI_WARPS], 1ull);
             }
             if constexpr (!GRID) {
-                if (rot_ok) {
-                    // bound: k list entries pairwise farther than 2*rho apart.
-                    // Loops over the register list are fully unrolled (static indices keep it in registers).
-                    unsigned long long Tw = KEY_MAX;
-                    uint32_t chosen[32];
-                    int nc = 0;
-#pragma unroll
-                    for (int i = 0; i < LIST; i++) {
-                        const unsigned long long key = lst[i];
-                        if (key != KEY_MAX && nc < a.k) {
-                            const uint32_t t = static_cast<uint32_t>(key & 0xffffffffu);
-                            bool far = true;
-                            for (int c = 0; c < nc; c++)
-                                far = far && dk::cheb_cyc(t, chosen[c], a.nx, a.ny, a.nz) > 2 * a.rho;
-                            if (far) {
-                                chosen[nc] = t;
-                                nc++;
-                                if (nc == a.k) Tw = key;
-                            }
-                        }
-                    }
-                    const unsigned long long old = atomicMin(&a.T[slot], Tw);
-                    const unsigned long long Tn = old < Tw ? old : Tw;
-                    atomicMin(&a.mu[slot], lst[LIST - 1]);
-#pragma unroll
-                    for (int i = 0; i < LIST; i++) {
-                        const unsigned long long key = lst[i];
-                        if (key != KEY_MAX && key <= Tn) {
-                            const unsigned pos = atomicAdd(&a.cnt[slot], 1u);
-                            if (pos < static_cast<unsigned>(a.cap)) a.cand[static_cast<size_t>(slot) * a.cap + pos] = key;
-                        }
-                    }
-                }
+                if (rot_ok) epi_publish(lst, slot, a);
             }
         }
     }
     tc_fence_before();
     __syncthreads();
     if (warp == 1) asm volatile("tcgen05.dealloc.cta_group::1.sync.aligned.b32 %0, 512;" ::"r"(tmem));
-    if constexpr (CL > 1) cluster_sync_all();
+}
+
+// ------------------------------------------------------------------ variant 2: streamed receptor planes
+//
+// Any number of channel groups G (P <= 32) and any probe size m <= 8, PAIR scheme per group, NTT
+// translations per MMA row (NTT = 64, 128 or 160 chosen at init to fit nx with the least waste) and Q
+// rows per tile (Q * NTT <= 512 TMEM columns).  K is walked unit by unit, unit u = (g, vz): the main
+// z-plane box of group g ((hi, lo) voxels, pass 1, M * MXP K-steps over (vy, vxp)) and its pair z-plane
+// box ((hi(x), hi(x+1)) slots, pass 2, M * MXQ K-steps over (vy, vxq)), padded to whole ring stages.
+// The two planes of a unit share one slot of an NR-deep receptor ring (one TMA box each, one barrier
+// pair per slot), so shared memory holds NR units whatever G and m are -- this is what lets the
+// large configuration (P = 22, m = 8) run on the tensor cores.
+__host__ __device__ constexpr int unit_ksteps(int m) { return m * ((m + 1) / 2) + m * ((m + 3) / 4); }
+__host__ __device__ constexpr int unit_ksteps_padded(int m) { return (unit_ksteps(m) + KSTEPS - 1) / KSTEPS * KSTEPS; }
+__host__ __device__ constexpr uint32_t stream_plane_stride(int m, int ntt, int q)
+{
+    return (static_cast<uint32_t>(q + m - 1) * static_cast<uint32_t>(pair_txb(m, ntt)) * 16u + 127u) / 128u * 128u;
+}
+// byte offset of K-step s of a unit inside its slot (main plane at 0, pair plane at pstride)
+__host__ __device__ constexpr uint32_t unit_off(int m, int s, uint32_t row16, uint32_t pstride)
+{
+    const int mxp = (m + 1) / 2, mxq = (m + 3) / 4, kp1 = m * mxp, kp2 = m * mxq;
+    return s < kp1        ? static_cast<uint32_t>(s / mxp) * row16 + static_cast<uint32_t>(s % mxp) * 32u
+           : s < kp1 + kp2 ? pstride + static_cast<uint32_t>((s - kp1) / mxq) * row16 +
+                                static_cast<uint32_t>((s - kp1) % mxq) * 64u
+                          : 0u;   // padding step: zero weights, any finite receptor data
+}
+
+template <int M, int NTT, int Q, bool GRID>
+__global__ void __launch_bounds__(NTHREADS, 1) k_corr_tcs(const __grid_constant__ CUtensorMap tmap,
+                                                           const __grid_constant__ CUtensorMap tmap_pair,
+                                                           const TcArgs a)
+{
+    constexpr int KS = KSTEPS;
+    constexpr unsigned STAGE = KS * WCHUNK;
+    constexpr int MXP = (M + 1) / 2;
+    constexpr int KP1 = M * MXP;                  // pass-1 K-steps of a unit
+    constexpr int KU = unit_ksteps(M);
+    constexpr int KUP = unit_ksteps_padded(M);
+    constexpr int NSU = KUP / KS;                 // weight stages per unit
+    constexpr uint32_t ROW16 = static_cast<uint32_t>(pair_txb(M, NTT)) * 16u;
+    constexpr uint32_t PLANE = static_cast<uint32_t>(Q + M - 1) * ROW16;   // bytes of one z-plane box
+    constexpr uint32_t PSTRIDE = stream_plane_stride(M, NTT, Q);
+    constexpr int NRMAX = 4;
+    static_assert(Q * NTT <= 512, "TMEM has 512 columns");
+    static_assert(NTT % 32 == 0 && NTT >= 32 && NTT <= 256, "MMA N");
+    extern __shared__ __align__(1024) unsigned char smem[];
+    __shared__ uint64_t bars[2 * NRMAX + 2 * WSTAGES + 1 + Q];
+    __shared__ uint32_t tmem_base_s;
+    uint64_t* rec_full = bars;
+    uint64_t* rec_empty = bars + NRMAX;
+    uint64_t* w_full = bars + 2 * NRMAX;
+    uint64_t* w_empty = w_full + WSTAGES;
+    uint64_t* tm_full = w_empty + WSTAGES;
+    uint64_t* tm_empty = tm_full + 1;   // [Q]
+
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    const int block = blockIdx.x / a.G, region = blockIdx.x % a.G;
+    const int tile_begin = region * a.tiles_per_region;
+    const int tile_end = min(a.ntiles, tile_begin + a.tiles_per_region);
+    const int n_tiles = tile_end - tile_begin;
+    const int NU = a.G_ch * M;          // units per tile
+    const int NR = a.n_rec_stages;      // receptor ring depth (units)
+    unsigned char* rec_smem = smem;     // [NR][slot = main plane | pair plane]
+    unsigned char* w_smem = smem + NR * a.rec_stage_bytes;
+
+    if (threadIdx.x == 0) {
+        for (int i = 0; i < NR; i++) {
+            dk::mbar_init(&rec_full[i], 1);
+            dk::mbar_init(&rec_empty[i], 1);
+        }
+        for (int i = 0; i < a.wstages; i++) {
+            dk::mbar_init(&w_full[i], 1);
+            dk::mbar_init(&w_empty[i], 1);
+        }
+        dk::mbar_init(&tm_full[0], 1);
+        for (int i = 0; i < Q; i++) dk::mbar_init(&tm_empty[i], a.nepi);
+        dk::fence_mbar_init();
+    }
+    if (warp == 1) {
+        asm volatile("tcgen05.alloc.cta_group::1.sync.aligned.shared::cta.b32 [%0], 512;" ::"r"(
+            dk::smem_u32(&tmem_base_s)));
+        asm volatile("tcgen05.relinquish_alloc_permit.cta_group::1.sync.aligned;");
+    }
+    tc_fence_before();
+    __syncthreads();
+    tc_fence_after();
+    const uint32_t tmem = tmem_base_s;
+
+    const bool tr = a.trace != nullptr;
+    long long tw0 = 0, tw1 = 0, tw2 = 0, tstart = tr ? clock64() : 0;
+    if (n_tiles > 0) {
+        if (warp == 0) {
+            // ------------------------------------------------ TMA producer (one thread), in unit order:
+            // the unit's two planes into the next receptor slot, then its weight stages into the ring
+            if (elect_one()) {
+                dk::prefetch_tmap(&tmap);
+                dk::prefetch_tmap(&tmap_pair);
+                const unsigned char* wsrc = a.W + static_cast<size_t>(block) * a.nsteps * WCHUNK;
+                int ws = 0, wph = 0, wuse = 0;
+                int rs = 0, rph = 0, ruse = 0;
+                int tx = tile_begin % a.ntx, ty = (tile_begin / a.ntx) % a.nty, tz = tile_begin / (a.ntx * a.nty);
+                for (int ti = 0; ti < n_tiles; ti++) {
+                    for (int u = 0; u < NU; u++) {
+                        const int g = u / M, vz = u % M;
+                        if (ruse >= NR) twait(&rec_empty[rs], rph ^ 1, tr, tw1);
+                        unsigned char* dst = rec_smem + static_cast<size_t>(rs) * a.rec_stage_bytes;
+                        dk::mbar_arrive_expect_tx(&rec_full[rs], 2 * PLANE);
+                        tma_load_5d(dst, &tmap, 0, tx * NTT, ty * Q, tz + vz, g, &rec_full[rs]);
+                        tma_load_5d(dst + PSTRIDE, &tmap_pair, 0, tx * NTT, ty * Q, tz + vz, g, &rec_full[rs]);
+                        ruse++;
+                        if (++rs == NR) {
+                            rs = 0;
+                            rph ^= 1;
+                        }
+                        const unsigned char* wu = wsrc + static_cast<size_t>(u) * KUP * WCHUNK;
+                        for (int st = 0; st < NSU; st++) {
+                            if (wuse >= a.wstages) twait(&w_empty[ws], wph ^ 1, tr, tw0);
+                            dk::mbar_arrive_expect_tx(&w_full[ws], STAGE);
+                            dk::bulk_load(w_smem + static_cast<size_t>(ws) * STAGE,
+                                          wu + static_cast<size_t>(st) * STAGE, STAGE, &w_full[ws]);
+                            wuse++;
+                            if (++ws == a.wstages) {
+                                ws = 0;
+                                wph ^= 1;
+                            }
+                        }
+                    }
+                    if (++tx == a.ntx) {
+                        tx = 0;
+                        if (++ty == a.nty) {
+                            ty = 0;
+                            tz++;
+                        }
+                    }
+                }
+                if (tr) {
+                    atomicAdd(&a.trace[TR_PROD_TOTAL], static_cast<unsigned long long>(clock64() - tstart));
+                    atomicAdd(&a.trace[TR_PROD_WEMPTY], static_cast<unsigned long long>(tw0));
+                    atomicAdd(&a.trace[TR_PROD_REMPTY], static_cast<unsigned long long>(tw1));
+                    atomicAdd(&a.trace[TR_CTAS], 1ull);
+                    atomicAdd(&a.trace[TR_TILES], static_cast<unsigned long long>(n_tiles));
+                }
+            }
+            __syncwarp();
+        } else if (warp == 1) {
+            // ------------------------------------------------ MMA issuer (one thread); the stage loop of a
+            // unit is unrolled so every in-slot descriptor offset is an immediate
+            constexpr uint32_t idesc = umma_idesc(ROT, NTT);
+            const uint32_t rec0 = dk::smem_u32(rec_smem), w0 = dk::smem_u32(w_smem);
+            const uint64_t dA0 = umma_desc(w0, ROT * 16, 128);
+            const uint64_t dB0 = umma_desc(rec0, 16, 128);   // pass 1: chunk LBO 16 B (voxel vx + 1)
+            const uint64_t dP0 = umma_desc(rec0, 32, 128);   // pass 2: chunk LBO 32 B (slot x + 2)
+            if (elect_one()) {
+                uint32_t ws = 0, wph = 0;
+                const uint32_t nws = static_cast<uint32_t>(a.wstages);
+                int rs = 0, rph = 0;
+                for (int ti = 0; ti < n_tiles; ti++) {
+                    for (int u = 0; u < NU; u++) {
+                        twait(&rec_full[rs], rph, tr, tw2);
+                        tc_fence_after();
+                        const uint32_t rofs = static_cast<uint32_t>(rs * a.rec_stage_bytes);
+                        const uint64_t dB = dB0 + (rofs >> 4), dP = dP0 + (rofs >> 4);
+#pragma unroll
+                        for (int st = 0; st < NSU; st++) {
+                            twait(&w_full[ws], wph, tr, tw1);
+                            tc_fence_after();
+                            const uint64_t da0 = dA0 + ((ws * STAGE) >> 4);
+                            if (st == 0 && u == 0 && ti > 0) {
+                                // first stage of a tile: each accumulator row restarts once the epilogue
+                                // released it
+#pragma unroll
+                                for (int q = 0; q < Q; q++) {
+                                    twait(&tm_empty[q], (ti - 1) & 1, tr, tw0);
+                                    tc_fence_after();
+#pragma unroll
+                                    for (int ks = 0; ks < KS; ks++)
+                                        umma_bf16(tmem + q * NTT, da0 + ((ks * WCHUNK) >> 4),
+                                                  (ks < KP1 || ks >= KU ? dB : dP) +
+                                                      ((unit_off(M, ks, ROW16, PSTRIDE) + q * ROW16) >> 4),
+                                                  idesc, ks == 0 ? 0u : 1u);
+                                }
+                            } else {
+                                const bool first = st == 0 && u == 0;   // ti == 0 here
+#pragma unroll
+                                for (int ks = 0; ks < KS; ks++) {
+                                    const int s = st * KS + ks;
+#pragma unroll
+                                    for (int q = 0; q < Q; q++)
+                                        umma_bf16(tmem + q * NTT, da0 + ((ks * WCHUNK) >> 4),
+                                                  (s < KP1 || s >= KU ? dB : dP) +
+                                                      ((unit_off(M, s, ROW16, PSTRIDE) + q * ROW16) >> 4),
+                                                  idesc, (first && ks == 0) ? 0u : 1u);
+                                }
+                            }
+                            umma_commit(&w_empty[ws]);
+                            if (++ws == nws) {
+                                ws = 0;
+                                wph ^= 1;
+                            }
+                        }
+                        umma_commit(&rec_empty[rs]);
+                        if (++rs == a.n_rec_stages) {
+                            rs = 0;
+                            rph ^= 1;
+                        }
+                    }
+                    umma_commit(&tm_full[0]);
+                }
+                if (tr) {
+                    atomicAdd(&a.trace[TR_MMA_TOTAL], static_cast<unsigned long long>(clock64() - tstart));
+                    atomicAdd(&a.trace[TR_MMA_TMEMPTY], static_cast<unsigned long long>(tw0));
+                    atomicAdd(&a.trace[TR_MMA_WFULL], static_cast<unsigned long long>(tw1));
+                    atomicAdd(&a.trace[TR_MMA_RFULL], static_cast<unsigned long long>(tw2));
+                }
+            }
+            __syncwarp();
+        } else {
+            // ------------------------------------------------ epilogue warps
+            const int quarter = warp & 3;
+            const int cls = (warp - 2) >> 2;
+            const int nclass = a.nepi >> 2;
+            const int r = quarter * 32 + lane;
+            const int slot = block * ROT + r;
+            const bool rot_ok = slot < a.n_slots;
+            unsigned long long lst[LIST];
+#pragma unroll
+            for (int i = 0; i < LIST; i++) lst[i] = KEY_MAX;
+            float th = __int_as_float(0x7f800000);
+            uint32_t th_t = 0xffffffffu;
+            int tx = tile_begin % a.ntx, ty = (tile_begin / a.ntx) % a.nty, tz = tile_begin / (a.ntx * a.nty);
+            for (int ti = 0; ti < n_tiles; ti++) {
+                twait(&tm_full[0], ti & 1, tr, tw0);
+                tc_fence_after();
+                epi_tile<NTT, Q, GRID>(a, tmem, tm_empty, quarter, cls, nclass, lane, slot, rot_ok, tx, ty, tz, lst,
+                                       th, th_t, tr, tw1);
+                if (++tx == a.ntx) {
+                    tx = 0;
+                    if (++ty == a.nty) {
+                        ty = 0;
+                        tz++;
+                    }
+                }
+            }
+            if (tr && lane == 0) {
+                atomicAdd(&a.trace[TR_EPI_TOTAL], static_cast<unsigned long long>(clock64() - tstart));
+                atomicAdd(&a.trace[TR_EPI_TMFULL], static_cast<unsigned long long>(tw0));
+                atomicAdd(&a.trace[TR_EPI_LDTM], static_cast<unsigned long long>(tw1));
+                atomicAdd(&a.trace[TR_EPI_WARPS], 1ull);
+            }
+            if constexpr (!GRID) {
+                if (rot_ok) epi_publish(lst, slot, a);
+            }
+        }
+    }
+    tc_fence_before();
+    __syncthreads();
+    if (warp == 1) asm volatile("tcgen05.dealloc.cta_group::1.sync.aligned.b32 %0, 512;" ::"r"(tmem));
 }
 
 // ------------------------------------------------------------------ data preparation
 
 // bf16 split of the padded receptor: Rb[g][Z][Y][X][8] = (hi_0..3, lo_0..3) of channels 4g..4g+3
+#ifndef DOCK_LAUNCHER_TU   // defined once, in dock.cu
 __global__ void k_pack_receptor_tc(const float* __restrict__ R, uint16_t* __restrict__ Rb, int nx, int ny, int nz,
                                    int Xp, int Yp, int Zp, int P, int G_ch)
 {
@@ -776,66 +869,26 @@ __global__ void k_pack_receptor_tc(const float* __restrict__ R, uint16_t* __rest
         reinterpret_cast<uint4*>(Rb)[i] = pk;
     }
 }
+#endif
 
-// Folded weights Lw [batch][P][m^3][RB] (k_voxelize output) -> A operand [block][step][chunk][rot][8].
-__global__ void k_pack_weights_tc(const float* __restrict__ Lw, unsigned char* __restrict__ W, int n_slots, int P,
-                                  int G_ch, int m, int nsteps)
-{
-    const int MXP = (m + 1) / 2, m3 = m * m * m;
-    const long long n_blocks = (n_slots + ROT - 1) / ROT;
-    const long long total = n_blocks * nsteps * 2 * ROT;   // one thread per (block, step, chunk, rot) 16-B row
-    for (long long i = blockIdx.x * static_cast<long long>(blockDim.x) + threadIdx.x; i < total;
-         i += static_cast<long long>(gridDim.x) * blockDim.x) {
-        const int r = static_cast<int>(i % ROT);
-        const int c = static_cast<int>((i / ROT) % 2);
-        const int s = static_cast<int>((i / (2 * ROT)) % nsteps);
-        const long long blk = i / (2LL * ROT * nsteps);
-        const int vxp = s % MXP, vy = (s / MXP) % m, vz = (s / (MXP * m)) % m;
-        const int pass = (s / (MXP * m * m)) % 2, g = s / (MXP * m * m * 2);
-        const int vx = 2 * vxp + c;
-        const long long slot = blk * ROT + r;
-        uint16_t out[8] = {0, 0, 0, 0, 0, 0, 0, 0};
-        if (slot < n_slots && vx < m) {
-            const int v = (vz * m + vy) * m + vx;
-#pragma unroll
-            for (int cc = 0; cc < 4; cc++) {
-                const int p = 4 * g + cc;
-                if (p >= P) continue;
-                const float f = Lw[((static_cast<size_t>(slot / dk::RB) * P + p) * m3 + v) * dk::RB + slot % dk::RB];
-                const __nv_bfloat16 hi = __float2bfloat16_rn(f);
-                const __nv_bfloat16 lo = __float2bfloat16_rn(f - __bfloat162float(hi));
-                if (pass == 0) {
-                    out[cc] = __bfloat16_as_ushort(hi);
-                    out[4 + cc] = __bfloat16_as_ushort(hi);
-                } else {
-                    out[cc] = __bfloat16_as_ushort(lo);
-                }
-            }
-        }
-        uint4 pk;
-        pk.x = out[0] | (static_cast<uint32_t>(out[1]) << 16);
-        pk.y = out[2] | (static_cast<uint32_t>(out[3]) << 16);
-        pk.z = out[4] | (static_cast<uint32_t>(out[5]) << 16);
-        pk.w = out[6] | (static_cast<uint32_t>(out[7]) << 16);
-        reinterpret_cast<uint4*>(W)[i] = pk;
-    }
-}
-
-// PAIR scheme, second receptor copy: slot X holds (Rhi_0..3(X), Rhi_0..3(X+1)) of channels 0..3.
+// PAIR scheme, second receptor copy: Rp[g][Z][Y][X][8] = (Rhi_{4g..4g+3}(X), Rhi_{4g..4g+3}(X+1)).
+#ifndef DOCK_LAUNCHER_TU   // defined once, in dock.cu
 __global__ void k_pack_receptor_pair_tc(const float* __restrict__ R, uint16_t* __restrict__ Rb, int nx, int ny, int nz,
-                                        int Xp, int Yp, int Zp, int P)
+                                        int Xp, int Yp, int Zp, int P, int G_ch)
 {
-    const size_t total = static_cast<size_t>(Zp) * Yp * Xp;
+    const size_t total = static_cast<size_t>(G_ch) * Zp * Yp * Xp;
     for (size_t i = blockIdx.x * static_cast<size_t>(blockDim.x) + threadIdx.x; i < total;
          i += static_cast<size_t>(gridDim.x) * blockDim.x) {
         const int X = static_cast<int>(i % Xp);
         size_t rr = i / Xp;
         const int Y = static_cast<int>(rr % Yp);
-        const int Z = static_cast<int>(rr / Yp);
+        rr /= Yp;
+        const int Z = static_cast<int>(rr % Zp);
+        const int g = static_cast<int>(rr / Zp);
         uint16_t out[8];
 #pragma unroll
         for (int c = 0; c < 8; c++) {
-            const int p = c & 3, dx = c >> 2;
+            const int p = 4 * g + (c & 3), dx = c >> 2;
             float f = 0.f;
             if (p < P) f = R[((static_cast<size_t>(p) * nz + Z % nz) * ny + Y % ny) * nx + (X + dx) % nx];
             out[c] = __bfloat16_as_ushort(__float2bfloat16_rn(f));
@@ -848,9 +901,11 @@ __global__ void k_pack_receptor_pair_tc(const float* __restrict__ R, uint16_t* _
         reinterpret_cast<uint4*>(Rb)[i] = pk;
     }
 }
+#endif
 
 // PAIR scheme A operand: steps [0, S1p) = pass 1 chunks (Whi(vx), Whi(vx)), vx = 2 vxp + c;
 // steps [S1p, S1p + S2p) = pass 2 chunks (Wlo(vx0), Wlo(vx0 + 1)), vx0 = 4 vxq + 2c; padding = 0.
+#ifndef DOCK_LAUNCHER_TU   // defined once, in dock.cu
 __global__ void k_pack_weights_tc_pair(const float* __restrict__ Lw, unsigned char* __restrict__ W, int n_slots, int P,
                                        int m, int S1, int S1p, int S2, int S2p)
 {
@@ -903,390 +958,64 @@ __global__ void k_pack_weights_tc_pair(const float* __restrict__ Lw, unsigned ch
         reinterpret_cast<uint4*>(W)[i] = pk;
     }
 }
+#endif
 
-// ------------------------------------------------------------------ variant 3: cta_group::2
-
-__device__ __forceinline__ void umma_bf16_2sm(uint32_t d_tmem, uint64_t a, uint64_t b, uint32_t idesc, uint32_t acc)
+// Streamed-plane A operand (variant 2): steps [u * KUP, (u + 1) * KUP) belong to unit u = (g, vz);
+// within a unit, steps [0, m * MXP) are pass-1 chunks (Whi(vx), Whi(vx)) over (vy, vxp), vx = 2 vxp + c,
+// steps [m * MXP, m * MXP + m * MXQ) pass-2 chunks (Wlo(vx0), Wlo(vx0 + 1)) over (vy, vxq),
+// vx0 = 4 vxq + 2c, of channels 4g..4g+3; the rest is zero padding.
+#ifndef DOCK_LAUNCHER_TU   // defined once, in dock.cu
+__global__ void k_pack_weights_tcs(const float* __restrict__ Lw, unsigned char* __restrict__ W, int n_slots, int P,
+                                   int m, int nsteps)
 {
-    asm volatile(
-        "{\n\t.reg .pred p;\n\tsetp.ne.b32 p, %4, 0;\n\t"
-        "tcgen05.mma.cta_group::2.kind::f16 [%0], %1, %2, %3, p;\n\t}\n" ::"r"(d_tmem),
-        "l"(a), "l"(b), "r"(idesc), "r"(acc)
-        : "memory");
-}
-__device__ __forceinline__ void umma_commit_2sm_mc(uint64_t* bar, uint16_t mask)
-{
-    asm volatile(
-        "tcgen05.commit.cta_group::2.mbarrier::arrive::one.shared::cluster.multicast::cluster.b64 [%0], %1;" ::"r"(
-            dk::smem_u32(bar)),
-        "h"(mask)
-        : "memory");
-}
-// Arrive on the barrier at the same shared-memory offset in CTA `rank` of the cluster.
-__device__ __forceinline__ void mbar_arrive_remote(uint64_t* bar, uint32_t rank)
-{
-    asm volatile(
-        "{\n\t.reg .b32 ra;\n\tmapa.shared::cluster.u32 ra, %0, %1;\n\t"
-        "mbarrier.arrive.release.cluster.shared::cluster.b64 _, [ra];\n\t}\n" ::"r"(dk::smem_u32(bar)),
-        "r"(rank)
-        : "memory");
-}
-
-// Variant 3: a CTA pair runs 256 rotations (its two blocks) against 4 receptor rows per tile,
-// each CTA holding 2 of the rows.  The leader issues tcgen05.mma.cta_group::2 M = 256 x N = 256:
-// A = each CTA's own 128 rotations, B = CTA0's row q (N 0..127) and CTA1's row q (N 128..255),
-// D = each CTA's TMEM [128 rotations][2 accumulators x 256 columns].  Per SM this halves the
-// shared-memory operand reads and the MMA instructions of variant 1.  Loads complete on local
-// barriers; the peer's MMA warp relays "stage full" to the leader with a remote arrive, and the
-// leader's commits release stages in both CTAs (multicast).
-template <int M, bool GRID>
-__global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc2(const __grid_constant__ CUtensorMap tmap,
-                                                           const __grid_constant__ CUtensorMap tmap_pair, const TcArgs a)
-{
-    constexpr int KS = KSTEPS;
-    constexpr unsigned STAGE = KS * WCHUNK;
-    constexpr int QL = 2;                 // receptor rows per CTA per tile; the pair covers 4
-    constexpr int MXP = (M + 1) / 2, MXQ = (M + 3) / 4;
-    extern __shared__ __align__(1024) unsigned char smem[];
-    __shared__ uint64_t bars[2 * 2 + 2 * WSTAGES + 2 + 2 + WSTAGES];
-    __shared__ uint32_t tmem_base_s;
-    uint64_t* rec_full = bars;
-    uint64_t* rec_empty = bars + 2;
-    uint64_t* w_full = bars + 4;
-    uint64_t* w_empty = w_full + WSTAGES;
-    uint64_t* tm_full = w_empty + WSTAGES;
-    uint64_t* tm_empty = tm_full + 1;
-    uint64_t* peer_rec = tm_empty + 1;    // leader only: peer's receptor buffers landed
-    uint64_t* peer_w = peer_rec + 2;      // leader only: peer's weight stages landed
-
-    uint32_t crank;
-    asm volatile("mov.u32 %0, %%cluster_ctarank;" : "=r"(crank));
-    const bool leader = crank == 0;
-    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
-    const int pitem = blockIdx.x >> 1;
-    const int bp = pitem / a.G, region = pitem % a.G;
-    const int block = 2 * bp + static_cast<int>(crank);
-    const int tile_begin = region * a.tiles_per_region;
-    const int tile_end = min(a.ntiles, tile_begin + a.tiles_per_region);
-    const int n_tiles = tile_end - tile_begin;
-    unsigned char* rec_smem = smem;
-    unsigned char* w_smem = smem + 2 * a.rec_stage_bytes;
-
-    if (threadIdx.x == 0) {
-        for (int i = 0; i < 2; i++) {
-            dk::mbar_init(&rec_full[i], 1);
-            dk::mbar_init(&rec_empty[i], 1);
-            dk::mbar_init(&peer_rec[i], 1);
-        }
-        for (int i = 0; i < a.wstages; i++) {
-            dk::mbar_init(&w_full[i], 1);
-            dk::mbar_init(&w_empty[i], 1);
-            dk::mbar_init(&peer_w[i], 1);
-        }
-        dk::mbar_init(&tm_full[0], 1);
-        dk::mbar_init(&tm_empty[0], 2 * a.nepi);
-        dk::fence_mbar_init();
-    }
-    if (warp == 1) {
-        asm volatile("tcgen05.alloc.cta_group::2.sync.aligned.shared::cta.b32 [%0], 512;" ::"r"(
-            dk::smem_u32(&tmem_base_s)));
-        asm volatile("tcgen05.relinquish_alloc_permit.cta_group::2.sync.aligned;");
-    }
-    tc_fence_before();
-    __syncthreads();
-    cluster_sync_all();
-    tc_fence_after();
-    const uint32_t tmem = tmem_base_s;
-    const bool tr = a.trace != nullptr;
-    long long tw0 = 0, tw1 = 0, tw2 = 0, tstart = tr ? clock64() : 0;
-
-    if (n_tiles > 0) {
-        if (warp == 0) {
-            // ------------------------------------------------ TMA producer (both CTAs, local data)
-            if (elect_one()) {
-                dk::prefetch_tmap(&tmap);
-                dk::prefetch_tmap(&tmap_pair);
-            }
-            const unsigned char* wsrc = a.W + static_cast<size_t>(block) * a.nsteps * WCHUNK;
-            int ws = 0, wph = 0, wuse = 0;
-            auto stream_weights = [&](int s0, int s1) {
-                for (int s = s0; s < s1; s += KS) {
-                    if (wuse >= a.wstages) twait(&w_empty[ws], wph ^ 1, tr, tw0);
-                    if (elect_one()) {
-                        dk::mbar_arrive_expect_tx(&w_full[ws], STAGE);
-                        dk::bulk_load(w_smem + static_cast<size_t>(ws) * STAGE, wsrc + static_cast<size_t>(s) * WCHUNK,
-                                      STAGE, &w_full[ws]);
-                    }
-                    __syncwarp();
-                    wuse++;
-                    if (++ws == a.wstages) {
-                        ws = 0;
-                        wph ^= 1;
-                    }
-                }
-            };
-            int pm = 0, pp = 0;
-            auto issue_box = [&](int which, int t) {
-                const int tile = tile_begin + t;
-                const int tx = tile % a.ntx, ty = (tile / a.ntx) % a.nty, tz = tile / (a.ntx * a.nty);
-                const int y0 = ty * (2 * QL) + QL * static_cast<int>(crank);
-                if (elect_one()) {
-                    dk::mbar_arrive_expect_tx(&rec_full[which], a.box_bytes);
-                    tma_load_5d(rec_smem + which * a.rec_stage_bytes, which ? &tmap_pair : &tmap, 0, tx * NT, y0, tz,
-                                0, &rec_full[which]);
-                }
-                __syncwarp();
-            };
-            auto poll = [&](int ti) {
-                if (pm < n_tiles && pm <= ti + 1 && (pm == 0 || dk::mbar_test(&rec_empty[0], (pm - 1) & 1)))
-                    issue_box(0, pm++);
-                if (pp < n_tiles && pp <= ti + 1 && (pp == 0 || dk::mbar_test(&rec_empty[1], (pp - 1) & 1)))
-                    issue_box(1, pp++);
-            };
-            auto ensure = [&](int which, int t) {
-                int& nx = which ? pp : pm;
-                if (nx == t) {
-                    if (t > 0) twait(&rec_empty[which], (t - 1) & 1, tr, tw1);
-                    issue_box(which, nx++);
-                }
-            };
-            for (int ti = 0; ti < n_tiles; ti++) {
-                ensure(0, ti);
-                for (int s = 0; s < a.S1p; s += KS) {
-                    poll(ti);
-                    stream_weights(s, s + KS);
-                }
-                ensure(1, ti);
-                for (int s = a.S1p; s < a.nsteps; s += KS) {
-                    poll(ti);
-                    stream_weights(s, s + KS);
-                }
-            }
-            if (tr && leader && elect_one()) {
-                atomicAdd(&a.trace[TR_PROD_TOTAL], static_cast<unsigned long long>(clock64() - tstart));
-                atomicAdd(&a.trace[TR_PROD_WEMPTY], static_cast<unsigned long long>(tw0));
-                atomicAdd(&a.trace[TR_PROD_REMPTY], static_cast<unsigned long long>(tw1));
-                atomicAdd(&a.trace[TR_CTAS], 1ull);
-                atomicAdd(&a.trace[TR_TILES], static_cast<unsigned long long>(n_tiles));
-            }
-            __syncwarp();
-        } else if (warp == 1) {
-            if (!leader) {
-                // ------------------------------------------------ relay: tell the leader our stages landed
-                int ws = 0, wph = 0;
-                auto relay_stages = [&](int n) {
-                    for (int s = 0; s < n; s += KS) {
-                        dk::mbar_wait(&w_full[ws], wph);
-                        if (elect_one()) mbar_arrive_remote(&peer_w[ws], 0);
-                        __syncwarp();
-                        if (++ws == a.wstages) {
-                            ws = 0;
-                            wph ^= 1;
-                        }
-                    }
-                };
-                for (int ti = 0; ti < n_tiles; ti++) {
-                    dk::mbar_wait(&rec_full[0], ti & 1);
-                    if (elect_one()) mbar_arrive_remote(&peer_rec[0], 0);
-                    __syncwarp();
-                    relay_stages(a.S1p);
-                    dk::mbar_wait(&rec_full[1], ti & 1);
-                    if (elect_one()) mbar_arrive_remote(&peer_rec[1], 0);
-                    __syncwarp();
-                    relay_stages(a.S2p);
-                }
-            } else {
-                // ------------------------------------------------ leader: MMA issue for the pair
-                constexpr uint32_t idesc = umma_idesc(2 * ROT, 2 * NT);
-                constexpr uint16_t PAIRMASK = 3;
-                const uint32_t rec0 = dk::smem_u32(rec_smem), w0 = dk::smem_u32(w_smem);
-                const uint64_t dA0 = umma_desc(w0, ROT * 16, 128);
-                const uint64_t dB0 = umma_desc(rec0, 16, 128);
-                const uint64_t dP0 = umma_desc(rec0 + a.rec_stage_bytes, 32, 128);
-                const uint32_t row16 = static_cast<uint32_t>(a.TXB) * 16u;
-                const uint32_t rowTY = static_cast<uint32_t>(a.TYB) * row16;
-                int ws = 0, wph = 0;
-                auto issue_stage = [&](int kind, int s0, bool first) {
-                    twait(&w_full[ws], wph, tr, tw1);
-                    twait(&peer_w[ws], wph, tr, tw1);
-                    tc_fence_after();
-                    if (elect_one()) {
-                        const uint64_t da0 = dA0 + ((static_cast<uint32_t>(ws) * STAGE) >> 4);
+    const int MXP = (m + 1) / 2, MXQ = (m + 3) / 4, m3 = m * m * m;
+    const int KP1 = m * MXP, KU = KP1 + m * MXQ, KUP = (KU + KSTEPS - 1) / KSTEPS * KSTEPS;
+    const long long n_blocks = (n_slots + ROT - 1) / ROT;
+    const long long total = n_blocks * nsteps * 2 * ROT;
+    for (long long i = blockIdx.x * static_cast<long long>(blockDim.x) + threadIdx.x; i < total;
+         i += static_cast<long long>(gridDim.x) * blockDim.x) {
+        const int r = static_cast<int>(i % ROT);
+        const int c = static_cast<int>((i / ROT) % 2);
+        const int s = static_cast<int>((i / (2 * ROT)) % nsteps);
+        const long long blk = i / (2LL * ROT * nsteps);
+        const long long slot = blk * ROT + r;
+        const int u = s / KUP, sl = s % KUP, g = u / m, vz = u % m;
+        uint16_t out[8] = {0, 0, 0, 0, 0, 0, 0, 0};
+        auto wval = [&](int vy, int vx, int p) -> float {
+            if (vx >= m || p >= P) return 0.f;
+            const int v = (vz * m + vy) * m + vx;
+            return Lw[((static_cast<size_t>(slot / dk::RB) * P + p) * m3 + v) * dk::RB + slot % dk::RB];
+        };
+        if (slot < n_slots) {
+            if (sl < KP1) {
+                const int vy = sl / MXP, vx = 2 * (sl % MXP) + c;
 #pragma unroll
-                        for (int ks = 0; ks < KS; ks++) {
-                            const int s = s0 + ks;
-                            uint64_t db;
-                            if (kind == 0) {
-                                const int vxp = s % MXP, vy = (s / MXP) % M, vz = s / (MXP * M);
-                                db = s < a.S1 ? dB0 + ((vz * rowTY + vy * row16 + vxp * 32u) >> 4) : dB0;
-                            } else {
-                                const int vxq = s % MXQ, vy = (s / MXQ) % M, vz = s / (MXQ * M);
-                                db = s < a.S2 ? dP0 + ((vz * rowTY + vy * row16 + vxq * 64u) >> 4) : dP0;
-                            }
-                            const uint64_t da = da0 + ((ks * WCHUNK) >> 4);
-#pragma unroll
-                            for (int q = 0; q < QL; q++)
-                                umma_bf16_2sm(tmem + q * 2 * NT, da, db + ((q * row16) >> 4), idesc,
-                                              (first && ks == 0) ? 0u : 1u);
-                        }
-                        umma_commit_2sm_mc(&w_empty[ws], PAIRMASK);
-                    }
-                    __syncwarp();
-                    if (++ws == a.wstages) {
-                        ws = 0;
-                        wph ^= 1;
-                    }
-                };
-                for (int ti = 0; ti < n_tiles; ti++) {
-                    twait(&rec_full[0], ti & 1, tr, tw2);
-                    twait(&peer_rec[0], ti & 1, tr, tw2);
-                    if (ti > 0) twait(&tm_empty[0], (ti - 1) & 1, tr, tw0);
-                    tc_fence_after();
-                    for (int s = 0; s < a.S1p; s += KS) issue_stage(0, s, s == 0);
-                    if (elect_one()) umma_commit_2sm_mc(&rec_empty[0], PAIRMASK);
-                    __syncwarp();
-                    twait(&rec_full[1], ti & 1, tr, tw2);
-                    twait(&peer_rec[1], ti & 1, tr, tw2);
-                    tc_fence_after();
-                    for (int s = 0; s < a.S2p; s += KS) issue_stage(1, s, false);
-                    if (elect_one()) {
-                        umma_commit_2sm_mc(&rec_empty[1], PAIRMASK);
-                        umma_commit_2sm_mc(&tm_full[0], PAIRMASK);
-                    }
-                    __syncwarp();
+                for (int cc = 0; cc < 4; cc++) {
+                    const __nv_bfloat16 hi = __float2bfloat16_rn(wval(vy, vx, 4 * g + cc));
+                    out[cc] = out[4 + cc] = __bfloat16_as_ushort(hi);
                 }
-                if (tr && elect_one()) {
-                    atomicAdd(&a.trace[TR_MMA_TOTAL], static_cast<unsigned long long>(clock64() - tstart));
-                    atomicAdd(&a.trace[TR_MMA_TMEMPTY], static_cast<unsigned long long>(tw0));
-                    atomicAdd(&a.trace[TR_MMA_WFULL], static_cast<unsigned long long>(tw1));
-                    atomicAdd(&a.trace[TR_MMA_RFULL], static_cast<unsigned long long>(tw2));
-                }
-                __syncwarp();
-            }
-        } else if (warp < 2 + a.nepi) {
-            // ------------------------------------------------ epilogue warps (both CTAs)
-            const int quarter = warp & 3;
-            const int cls = (warp - 2) >> 2;                 // 0..3 -> (accumulator q, CTA half)
-            const int nclass = a.nepi >> 2;
-            const int r = quarter * 32 + lane;
-            const int slot = block * ROT + r;
-            const bool rot_ok = slot < a.n_slots;
-            unsigned long long lst[LIST];
+            } else if (sl < KU) {
+                const int t = sl - KP1, vy = t / MXQ, vx0 = 4 * (t % MXQ) + 2 * c;
 #pragma unroll
-            for (int i = 0; i < LIST; i++) lst[i] = KEY_MAX;
-            float th = __int_as_float(0x7f800000);
-            uint32_t th_t = 0xffffffffu;
-            for (int ti = 0; ti < n_tiles; ti++) {
-                const int tile = tile_begin + ti;
-                twait(&tm_full[0], ti & 1, tr, tw0);
-                tc_fence_after();
-                if (a.dbg == 1) {   // diagnostic: no TMEM drain
-                    __syncwarp();
-                    if (lane == 0) {
-                        if (leader) dk::mbar_arrive(&tm_empty[0]);
-                        else mbar_arrive_remote(&tm_empty[0], 0);
-                    }
-                    continue;
-                }
-                const int tx = tile % a.ntx, ty = (tile / a.ntx) % a.nty, tz = tile / (a.ntx * a.nty);
-                for (int c4 = cls; c4 < 4; c4 += nclass) {
-                    const int q = c4 >> 1, half = c4 & 1;
-                    const int y = ty * (2 * QL) + QL * half + q, z = tz;
-                    const bool row_ok = rot_ok && y < a.ny && z < a.nz;
-                    const int x0 = tx * NT;
-                    const uint32_t tbase = static_cast<uint32_t>((z * a.ny + y) * a.nx + x0);
-#pragma unroll 1
-                    for (int c0 = 0; c0 < NT; c0 += 32) {
-                        uint32_t v[32];
-                        const long long tl0 = tr ? clock64() : 0;
-                        tmem_ld32(tmem + (static_cast<uint32_t>(quarter * 32) << 16) + q * 2 * NT + half * NT + c0, v);
-                        if (tr) tw1 += clock64() - tl0;
-                        if (!row_ok || a.dbg == 2) continue;
-                        if constexpr (GRID) {
-                            float* out = a.grid + static_cast<size_t>(slot) * a.nx * a.ny * a.nz + tbase;
+                for (int cc = 0; cc < 4; cc++) {
 #pragma unroll
-                            for (int j = 0; j < 32; j++)
-                                if (x0 + c0 + j < a.nx) out[c0 + j] = __uint_as_float(v[j]);
-                        } else {
-                            float mn = __uint_as_float(v[0]);
-#pragma unroll
-                            for (int j = 1; j < 32; j++) mn = fminf(mn, __uint_as_float(v[j]));
-                            if (mn < th || (mn == th && tbase + c0 < th_t)) {
-                                const int jmax = min(32, a.nx - x0 - c0);
-                                uint32_t msk = 0;
-#pragma unroll
-                                for (int j = 0; j < 32; j++)
-                                    msk |= (__uint_as_float(v[j]) <= th && j < jmax) ? (1u << j) : 0u;
-                                while (msk) {
-                                    const int j = __ffs(msk) - 1;
-                                    msk &= msk - 1;
-                                    const float sv = __uint_as_float(select32(v, j));
-                                    if (sv <= th) {
-                                        const unsigned long long key = dk::make_key(sv, tbase + c0 + j);
-                                        if (key < lst[LIST - 1]) {
-                                            list_insert(lst, key);
-                                            th = dk::key_score_bound(static_cast<uint32_t>(lst[LIST - 1] >> 32));
-                                            th_t = static_cast<uint32_t>(lst[LIST - 1] & 0xffffffffu);
-                                        }
-                                    }
-                                }
-                            }
-                        }
-                    }
-                }
-                tc_fence_before();
-                __syncwarp();
-                if (lane == 0) {
-                    if (leader) dk::mbar_arrive(&tm_empty[0]);
-                    else mbar_arrive_remote(&tm_empty[0], 0);
-                }
-            }
-            if (tr && leader && lane == 0) {
-                atomicAdd(&a.trace[TR_EPI_TOTAL], static_cast<unsigned long long>(clock64() - tstart));
-                atomicAdd(&a.trace[TR_EPI_TMFULL], static_cast<unsigned long long>(tw0));
-                atomicAdd(&a.trace[TR_EPI_LDTM], static_cast<unsigned long long>(tw1));
-                atomicAdd(&a.trace[TR_EPI_WARPS], 1ull);
-            }
-            if constexpr (!GRID) {
-                if (rot_ok) {
-                    unsigned long long Tw = KEY_MAX;
-                    uint32_t chosen[32];
-                    int nc = 0;
-#pragma unroll
-                    for (int i = 0; i < LIST; i++) {
-                        const unsigned long long key = lst[i];
-                        if (key != KEY_MAX && nc < a.k) {
-                            const uint32_t t = static_cast<uint32_t>(key & 0xffffffffu);
-                            bool far = true;
-                            for (int c = 0; c < nc; c++)
-                                far = far && dk::cheb_cyc(t, chosen[c], a.nx, a.ny, a.nz) > 2 * a.rho;
-                            if (far) {
-                                chosen[nc] = t;
-                                nc++;
-                                if (nc == a.k) Tw = key;
-                            }
-                        }
-                    }
-                    const unsigned long long old = atomicMin(&a.T[slot], Tw);
-                    const unsigned long long Tn = old < Tw ? old : Tw;
-                    atomicMin(&a.mu[slot], lst[LIST - 1]);
-#pragma unroll
-                    for (int i = 0; i < LIST; i++) {
-                        const unsigned long long key = lst[i];
-                        if (key != KEY_MAX && key <= Tn) {
-                            const unsigned pos = atomicAdd(&a.cnt[slot], 1u);
-                            if (pos < static_cast<unsigned>(a.cap)) a.cand[static_cast<size_t>(slot) * a.cap + pos] = key;
-                        }
+                    for (int d = 0; d < 2; d++) {
+                        const float f = wval(vy, vx0 + d, 4 * g + cc);
+                        const __nv_bfloat16 hi = __float2bfloat16_rn(f);
+                        const __nv_bfloat16 lo = __float2bfloat16_rn(f - __bfloat162float(hi));
+                        out[4 * d + cc] = __bfloat16_as_ushort(lo);
                     }
                 }
             }
         }
+        uint4 pk;
+        pk.x = out[0] | (static_cast<uint32_t>(out[1]) << 16);
+        pk.y = out[2] | (static_cast<uint32_t>(out[3]) << 16);
+        pk.z = out[4] | (static_cast<uint32_t>(out[5]) << 16);
+        pk.w = out[6] | (static_cast<uint32_t>(out[7]) << 16);
+        reinterpret_cast<uint4*>(W)[i] = pk;
     }
-    tc_fence_before();
-    __syncthreads();
-    cluster_sync_all();
-    if (warp == 1) asm volatile("tcgen05.dealloc.cta_group::2.sync.aligned.b32 %0, 512;" ::"r"(tmem));
-    cluster_sync_all();
 }
+#endif
 
 }  // namespace tc

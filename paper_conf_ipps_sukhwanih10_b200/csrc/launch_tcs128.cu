@@ -1,0 +1,23 @@
+// tcgen05 variant 2 instantiations (k_corr_tcs, dock_tc.cuh) for 128 translations per MMA row.
+#define DOCK_LAUNCHER_TU
+#include "dock_launch.h"
+
+template <int M, bool GRID>
+static cudaError_t launch_t(const CUtensorMap& tmap, const CUtensorMap& tmap_pair, int smem, const tc::TcArgs& a,
+                            int nblocks, cudaStream_t st)
+{
+    auto kern = tc::k_corr_tcs<M, 128, tcs_q(128), GRID>;
+    cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+    if (e != cudaSuccess) return e;
+    kern<<<nblocks, (2 + a.nepi) * 32, smem, st>>>(tmap, tmap_pair, a);
+    return cudaGetLastError();
+}
+
+cudaError_t dock_launch_tcs128(int m, bool grid, const CUtensorMap& tmap, const CUtensorMap& tmap_pair, int smem,
+                              const tc::TcArgs& a, int nblocks, cudaStream_t st)
+{
+#define CALL_G(M) launch_t<M, true>(tmap, tmap_pair, smem, a, nblocks, st)
+#define CALL_S(M) launch_t<M, false>(tmap, tmap_pair, smem, a, nblocks, st)
+    if (grid) { DOCK_DISPATCH_M(m, CALL_G) }
+    DOCK_DISPATCH_M(m, CALL_S)
+}

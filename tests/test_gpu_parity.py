@@ -26,12 +26,10 @@ def D():
     return D
 
 
-# engine ids used by the tests: 1 = FP32 FFMA; 2 = tcgen05 variant 1 (4 rows, 1 TMEM buffer);
-# 3 = tcgen05 variant 2 (2 rows, 2 TMEM buffers, CTA pair with multicast weights);
-# 4 = tcgen05 variant 3 (cta_group::2, M = 256 rotations x N = 256 translations over a CTA pair);
-# 5 = tcgen05 variant 4 (2 rows x 2 TMEM buffers, single CTA);
-# 6, 7 = tcgen05 variants 5, 6 (row-skewed schedule, z-plane receptor staging; 4 rows x 1 / 2 rows x 2 buffers)
-ENGINES = [1, 2, 3, 4, 5, 6, 7]
+# engine ids used by the tests: 1 = FP32 FFMA; 2 = tcgen05 variant 1 (one channel group, resident receptor
+# boxes, 128 translations x 4 rows); 3 = tcgen05 variant 2 (receptor streamed per (channel group, z-plane),
+# any P, 64 / 128 / 160 translations per row).  A tcgen05 variant that cannot run a case runs the other one.
+ENGINES = [1, 2, 3]
 
 
 def _ctx(D, R, w, m_max, engine=0):
@@ -88,6 +86,9 @@ def test_voxelize_matches_oracle(D, orc, m):
     ((37, 13, 9), 4, 2, "uniform"),     # lanes_x = 4 path, ragged everywhere
     ((40, 24, 24), 8, 3, "uniform"),    # largest probe grid
     ((33, 17, 19), 1, 1, "uniform"),    # m = 1
+    ((64, 12, 9), 4, 8, "ftmap"),       # two channel groups (variant 2, 64 translations x 8 rows)
+    ((160, 7, 6), 8, 22, "uniform"),    # large-config channels: six groups, 160 translations x 3 rows
+    ((96, 10, 7), 6, 13, "uniform"),    # four groups, ragged last group, 128-wide rows over nx = 96
 ])
 @pytest.mark.parametrize("engine", ENGINES)
 def test_score_grid_within_tolerance(D, orc, shape, m, P, kind, engine):
@@ -343,14 +344,16 @@ def test_prod_config_sampled(D, orc, engine):
     assert info["fallback_last"] <= 80 and _engine_id(info) == engine
 
 
-def test_large_config_sampled(D, orc):
+@pytest.mark.parametrize("engine", [1, 3])
+def test_large_config_sampled(D, orc, engine):
     """configs[4] shape: 160^3 receptor, 8^3 probe, 22 terms (pairwise-potential channels), k=4, rho=1.
-    A 256-rotation slice of the 70k-rotation set is docked on the GPU (the FFMA engine: the 22-channel
-    tcgen05 receptor box does not fit shared memory); two units are validated against the oracle."""
+    A 256-rotation slice of the 70k-rotation set is docked on the GPU (FFMA engine, and tcgen05 variant 2:
+    six channel groups streamed per z-plane, 160 translations per MMA row); two units are validated
+    against the oracle."""
     c = g.CONFIGS["large"]
     R = g.receptor_ftmap_like(c.n, c.P)
     w = g.weights(c.P)
     probes = g.probes(1, c.m, c.P)
     rot = g.rotations(256, seed=3001)
-    _, info, _ = _dock_and_validate(D, orc, R, w, probes, rot, c.k, 1, units=[0, 173])
-    assert info["fallback_last"] <= 4
+    _, info, _ = _dock_and_validate(D, orc, R, w, probes, rot, c.k, 1, units=[0, 173], engine=engine)
+    assert info["fallback_last"] <= 4 and _engine_id(info) == engine
