@@ -141,7 +141,8 @@ typedef enum {
                                      z-plane) unit at a time (any P <= 32, m <= 8; 64 / 128 / 160 translations per
                                      row, chosen at init for nx).  A variant that cannot run m falls back to the
                                      other one. */
-    DOCK_TUNE_TC_EPILOGUE_WARPS = 6 /* tcgen05 epilogue warps: 0 auto (one translation row per thread), 4, 8, 16 */
+    DOCK_TUNE_TC_EPILOGUE_WARPS = 6 /* tcgen05 epilogue warps: 0 auto (= the compiled maximum, 8), 4 or 8 (values
+                                     above the compiled maximum are clamped to it) */
 } dock_tune_key;
 
 dock_status dock_set_tuning(dock_ctx* ctx, int key, int64_t value);

@@ -48,7 +48,9 @@ def build_native(force: bool = False, verbose: bool = False) -> str:
 
     def compile_one(src_obj):
         src, obj = src_obj
-        cmd = [_nvcc(), *NVCC_FLAGS, "-I", os.path.join(ROOT, "include"), "-c", "-o", obj, src]
+        # DOCK_NVCC_DEFS: extra -D flags for tuning experiments (e.g. "-DDOCK_TC_STAIR=2"); unset in normal builds
+        extra = os.environ.get("DOCK_NVCC_DEFS", "").split()
+        cmd = [_nvcc(), *NVCC_FLAGS, *extra, "-I", os.path.join(ROOT, "include"), "-c", "-o", obj, src]
         return subprocess.run(cmd, capture_output=True, text=True)
 
     with ThreadPoolExecutor(max_workers=max(1, min(len(SOURCES), os.cpu_count() or 1))) as ex:

@@ -72,7 +72,7 @@ struct dock_ctx {
     int tc_variant_last = 0;
     int tc_m_last = 0;
     int tc_ksteps_last = 0;    // K-steps (of 16) per translation row in the last tcgen05 launch
-    int tc_nepi = 0;           // epilogue warps (0 = 16)
+    int tc_nepi = 0;           // epilogue warps (0 = tc::NEPI_MAX)
     uint16_t* d_rec_tc = nullptr;     // [g][Zp][Yp][Xp][8] bf16 (hi_0..3, lo_0..3)
     uint16_t* d_rec_pair = nullptr;   // [g][Zp][Yp][Xp][8] bf16 (hi_0..3(X), hi_0..3(X+1))
     int tc_Gch = 0, tc_Xp = 0, tc_Yp = 0, tc_Zp = 0;
@@ -607,7 +607,7 @@ tc::TcArgs tc_args(dock_ctx* ctx, int m, int v, int n_slots, int G, const unsign
     a.rec_stage_bytes = tp.rec_stage_bytes;
     a.n_rec_stages = tp.n_rec_stages;
     a.wstages = tp.wstages;
-    a.nepi = ctx->tc_nepi > 0 ? std::min(16, ctx->tc_nepi) : 16;
+    a.nepi = ctx->tc_nepi > 0 ? std::min(tc::NEPI_MAX, ctx->tc_nepi) : tc::NEPI_MAX;
     a.trace = ctx->d_trace;
     a.dbg = ctx->tc_dbg;
     return a;

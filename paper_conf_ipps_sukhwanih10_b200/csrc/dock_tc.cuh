@@ -32,7 +32,13 @@ using dk::KEY_MAX;
 
 constexpr int ROT = 128;        // rotations per block (MMA M)
 constexpr int NT = 128;         // translations per row (MMA N)
-constexpr int NEPI_MAX = 16;    // epilogue warps: a.nepi in {4, 8, 16} (1, 2 or 4 per TMEM lane quarter)
+#ifndef DOCK_TC_NEPI_MAX
+#define DOCK_TC_NEPI_MAX 8
+#endif
+#ifndef DOCK_TC_STAIR
+#define DOCK_TC_STAIR 3
+#endif
+constexpr int NEPI_MAX = DOCK_TC_NEPI_MAX;   // epilogue warps: a.nepi in {4, 8} (1 or 2 per TMEM lane quarter; 8 measured best: 168 registers per thread, 2 row classes)
 constexpr int NTHREADS = (2 + NEPI_MAX) * 32;   // launch bound; the launch uses (2 + a.nepi) * 32 threads
 constexpr int WSTAGES = 16;     // max weight ring depth (runtime a.wstages <= 16; 16 x 4 KB covers the L2 latency)
 constexpr int WCHUNK = 2 * ROT * 16;   // bytes of one K-step of A (2 K-chunks x 128 rotations x 16 B)
@@ -258,15 +264,21 @@ __device__ __forceinline__ void epi_publish(const unsigned long long (&lst)[LIST
 // registers, before that chunk is processed.  Within row q the warp takes the 32-column chunks
 // jj = cls, cls + nclass, ... at column ((q + jj) mod NCH) * 32 ("diagonal" classes: over the rows of a
 // tile a class's cells are spread like a row class).
+// row_full != nullptr: each row has its own "accumulated" barrier (parity row_ph), waited before its drain.
 template <int NTT, int Q, bool GRID>
 __device__ __forceinline__ void epi_tile(const TcArgs& a, uint32_t tmem, uint64_t* tm_empty, int quarter, int cls,
                                          int nclass, int lane, int slot, bool rot_ok, int tx, int ty, int tz,
                                          unsigned long long (&lst)[LIST], float& th, uint32_t& th_t, bool tr,
-                                         long long& tw1)
+                                         long long& tw0, long long& tw1, uint64_t* row_full = nullptr,
+                                         unsigned row_ph = 0)
 {
     constexpr int NCH = NTT / 32;
     const int x0 = tx * NTT;
     for (int q = 0; q < Q; q++) {
+        if (row_full) {
+            twait(&row_full[q], row_ph, tr, tw0);
+            tc_fence_after();
+        }
         const int y = ty * Q + q, z = tz;
         const bool row_ok = rot_ok && y < a.ny && z < a.nz;
         const uint32_t tbase = static_cast<uint32_t>((z * a.ny + y) * a.nx + x0);
@@ -340,14 +352,14 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
     constexpr uint32_t ROWTY = static_cast<uint32_t>(Q + M - 1) * ROW16;
     static_assert(Q * NT <= 512, "TMEM has 512 columns");
     extern __shared__ __align__(1024) unsigned char smem[];
-    __shared__ uint64_t bars[2 * 2 + 2 * WSTAGES + 1 + Q];
+    __shared__ uint64_t bars[2 * 2 + 2 * WSTAGES + 2 * Q];
     __shared__ uint32_t tmem_base_s;
     uint64_t* rec_full = bars;
     uint64_t* rec_empty = bars + 2;
     uint64_t* w_full = bars + 4;
     uint64_t* w_empty = w_full + WSTAGES;
-    uint64_t* tm_full = w_empty + WSTAGES;
-    uint64_t* tm_empty = tm_full + 1;   // [Q]: per accumulator row, so the next tile restarts row by row
+    uint64_t* tm_full = w_empty + WSTAGES;   // [Q]: row q accumulated (the staircase finishes rows one by one)
+    uint64_t* tm_empty = tm_full + Q;        // [Q]: row q drained, so the next tile restarts row by row
 
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     const int block = blockIdx.x / a.G, region = blockIdx.x % a.G;
@@ -366,8 +378,10 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
             dk::mbar_init(&w_full[i], 1);
             dk::mbar_init(&w_empty[i], 1);
         }
-        dk::mbar_init(&tm_full[0], 1);
-        for (int i = 0; i < Q; i++) dk::mbar_init(&tm_empty[i], a.nepi);
+        for (int i = 0; i < Q; i++) {
+            dk::mbar_init(&tm_full[i], 1);
+            dk::mbar_init(&tm_empty[i], a.nepi);
+        }
         dk::fence_mbar_init();
     }
     if (warp == 1) {
@@ -457,55 +471,73 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
             // ------------------------------------------------ MMA issuer (one thread runs the whole schedule)
             // The stage loops are unrolled so every descriptor offset is an immediate and the tcgen05 queue
             // stays fed (issuing per K-step from a converged warp capped the tensor pipe at 40-47 %).
+            // Staircase: the first D and the last D weight stages of a tile are issued row by row, so row q
+            // finishes (tm_full[q]) while rows q+1.. still compute and restarts as soon as the epilogue has
+            // drained it -- the TMEM drain (64 B/clk, a third of the MMA time at m = 4) overlaps the MMAs
+            // instead of stalling the tensor pipe at every tile boundary.
             constexpr uint32_t idesc = umma_idesc(ROT, NT);
+            constexpr int NS1 = S1P / KS, NS2 = S2P / KS;
+            constexpr int DS = DOCK_TC_STAIR;
+            constexpr int D = NS1 < NS2 ? (NS1 < DS ? NS1 : DS) : (NS2 < DS ? NS2 : DS);   // staircase depth
             const uint32_t rec0 = dk::smem_u32(rec_smem), w0 = dk::smem_u32(w_smem);
             const uint64_t dA0 = umma_desc(w0, ROT * 16, 128);                 // + (slot offset >> 4)
             const uint64_t dB0 = umma_desc(rec0, 16, 128);                     // + (voxel offset >> 4)
             const uint64_t dP0 = umma_desc(rec0 + a.rec_stage_bytes, 32, 128);
             if (elect_one()) {
-                uint32_t ws = 0, wph = 0;
+                uint32_t ws = 0, wph = 0;   // ring slot / phase of the next stage
                 const uint32_t nws = static_cast<uint32_t>(a.wstages);
-                for (int ti = 0; ti < n_tiles; ti++) {
-                    const uint32_t dcol = tmem;
-                    twait(&rec_full[0], ti & 1, tr, tw2);
-                    tc_fence_after();
-#pragma unroll
-                    for (int st = 0; st < S1P / KS; st++) {
-                        twait(&w_full[ws], wph, tr, tw1);
-                        tc_fence_after();
-                        const uint64_t da0 = dA0 + ((ws * STAGE) >> 4);
-                        if (st == 0 && ti > 0) {
-                            // accumulator rows are released one by one while the epilogue drains them
-#pragma unroll
-                            for (int q = 0; q < Q; q++) {
-                                twait(&tm_empty[q], (ti - 1) & 1, tr, tw0);
-                                tc_fence_after();
-#pragma unroll
-                                for (int ks = 0; ks < KS; ks++)
-                                    umma_bf16(dcol + q * NT, da0 + ((ks * WCHUNK) >> 4),
-                                              dB0 + ((pair_off1(M, ks, ROW16, ROWTY) + q * ROW16) >> 4), idesc,
-                                              ks == 0 ? 0u : 1u);
-                            }
-                        } else {
-#pragma unroll
-                            for (int ks = 0; ks < KS; ks++)
-#pragma unroll
-                                for (int q = 0; q < Q; q++)
-                                    umma_bf16(dcol + q * NT, da0 + ((ks * WCHUNK) >> 4),
-                                              dB0 + ((pair_off1(M, st * KS + ks, ROW16, ROWTY) + q * ROW16) >> 4),
-                                              idesc, (st == 0 && ks == 0) ? 0u : 1u);
-                        }
-                        umma_commit(&w_empty[ws]);
+                // slot and phase of the stage `ahead` stages after the next one
+                auto slot_of = [&](int ahead, uint32_t& ph) -> uint32_t {
+                    uint32_t sl = ws + static_cast<uint32_t>(ahead);
+                    ph = wph;
+                    if (sl >= nws) {
+                        sl -= nws;
+                        ph ^= 1u;
+                    }
+                    return sl;
+                };
+                auto advance = [&](int n) {
+                    for (int i = 0; i < n; i++)
                         if (++ws == nws) {
                             ws = 0;
                             wph ^= 1;
                         }
-                    }
-                    umma_commit(&rec_empty[0]);
-                    twait(&rec_full[1], ti & 1, tr, tw2);
+                };
+                for (int ti = 0; ti < n_tiles; ti++) {
+                    twait(&rec_full[0], ti & 1, tr, tw2);
                     tc_fence_after();
+                    // pass 1, stages [0, D): row by row, each row after the epilogue released it
 #pragma unroll
-                    for (int st = 0; st < S2P / KS; st++) {
+                    for (int q = 0; q < Q; q++) {
+                        if (ti > 0) {
+                            twait(&tm_empty[q], (ti - 1) & 1, tr, tw0);
+                            tc_fence_after();
+                        }
+#pragma unroll
+                        for (int st = 0; st < D; st++) {
+                            uint32_t ph;
+                            const uint32_t sl = slot_of(st, ph);
+                            if (q == 0) {
+                                twait(&w_full[sl], ph, tr, tw1);
+                                tc_fence_after();
+                            }
+                            const uint64_t da0 = dA0 + ((sl * STAGE) >> 4);
+#pragma unroll
+                            for (int ks = 0; ks < KS; ks++)
+                                umma_bf16(tmem + q * NT, da0 + ((ks * WCHUNK) >> 4),
+                                          dB0 + ((pair_off1(M, st * KS + ks, ROW16, ROWTY) + q * ROW16) >> 4), idesc,
+                                          (st == 0 && ks == 0) ? 0u : 1u);
+                        }
+                    }
+#pragma unroll
+                    for (int st = 0; st < D; st++) {
+                        uint32_t ph;
+                        umma_commit(&w_empty[slot_of(st, ph)]);
+                    }
+                    advance(D);
+                    // pass 1, stages [D, NS1): all rows per stage
+#pragma unroll
+                    for (int st = D; st < NS1; st++) {
                         twait(&w_full[ws], wph, tr, tw1);
                         tc_fence_after();
                         const uint64_t da0 = dA0 + ((ws * STAGE) >> 4);
@@ -513,17 +545,59 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                         for (int ks = 0; ks < KS; ks++)
 #pragma unroll
                             for (int q = 0; q < Q; q++)
-                                umma_bf16(dcol + q * NT, da0 + ((ks * WCHUNK) >> 4),
+                                umma_bf16(tmem + q * NT, da0 + ((ks * WCHUNK) >> 4),
+                                          dB0 + ((pair_off1(M, st * KS + ks, ROW16, ROWTY) + q * ROW16) >> 4), idesc,
+                                          1u);
+                        umma_commit(&w_empty[ws]);
+                        advance(1);
+                    }
+                    umma_commit(&rec_empty[0]);
+                    twait(&rec_full[1], ti & 1, tr, tw2);
+                    tc_fence_after();
+                    // pass 2, stages [0, NS2 - D): all rows per stage
+#pragma unroll
+                    for (int st = 0; st < NS2 - D; st++) {
+                        twait(&w_full[ws], wph, tr, tw1);
+                        tc_fence_after();
+                        const uint64_t da0 = dA0 + ((ws * STAGE) >> 4);
+#pragma unroll
+                        for (int ks = 0; ks < KS; ks++)
+#pragma unroll
+                            for (int q = 0; q < Q; q++)
+                                umma_bf16(tmem + q * NT, da0 + ((ks * WCHUNK) >> 4),
                                           dP0 + ((pair_off2(M, st * KS + ks, ROW16, ROWTY) + q * ROW16) >> 4), idesc,
                                           1u);
                         umma_commit(&w_empty[ws]);
-                        if (++ws == nws) {
-                            ws = 0;
-                            wph ^= 1;
-                        }
+                        advance(1);
                     }
+                    // pass 2, stages [NS2 - D, NS2): row by row; row q is complete after its block
+#pragma unroll
+                    for (int q = 0; q < Q; q++) {
+#pragma unroll
+                        for (int j = 0; j < D; j++) {
+                            const int st = NS2 - D + j;
+                            uint32_t ph;
+                            const uint32_t sl = slot_of(j, ph);
+                            if (q == 0) {
+                                twait(&w_full[sl], ph, tr, tw1);
+                                tc_fence_after();
+                            }
+                            const uint64_t da0 = dA0 + ((sl * STAGE) >> 4);
+#pragma unroll
+                            for (int ks = 0; ks < KS; ks++)
+                                umma_bf16(tmem + q * NT, da0 + ((ks * WCHUNK) >> 4),
+                                          dP0 + ((pair_off2(M, st * KS + ks, ROW16, ROWTY) + q * ROW16) >> 4), idesc,
+                                          1u);
+                        }
+                        umma_commit(&tm_full[q]);
+                    }
+#pragma unroll
+                    for (int j = 0; j < D; j++) {
+                        uint32_t ph;
+                        umma_commit(&w_empty[slot_of(j, ph)]);
+                    }
+                    advance(D);
                     umma_commit(&rec_empty[1]);
-                    umma_commit(&tm_full[0]);
                 }
                 if (tr) {
                     atomicAdd(&a.trace[TR_MMA_TOTAL], static_cast<unsigned long long>(clock64() - tstart));
@@ -548,10 +622,8 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
             uint32_t th_t = 0xffffffffu;             // t_lin of the list's last key
             int tx = tile_begin % a.ntx, ty = (tile_begin / a.ntx) % a.nty, tz = tile_begin / (a.ntx * a.nty);
             for (int ti = 0; ti < n_tiles; ti++) {
-                twait(&tm_full[0], ti & 1, tr, tw0);
-                tc_fence_after();
                 epi_tile<NT, Q, GRID>(a, tmem, tm_empty, quarter, cls, nclass, lane, slot, rot_ok, tx, ty, tz, lst, th,
-                                      th_t, tr, tw1);
+                                      th_t, tr, tw0, tw1, tm_full, ti & 1);
                 if (++tx == a.ntx) {
                     tx = 0;
                     if (++ty == a.nty) {
@@ -809,7 +881,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tcs(const __grid_constant_
                 twait(&tm_full[0], ti & 1, tr, tw0);
                 tc_fence_after();
                 epi_tile<NTT, Q, GRID>(a, tmem, tm_empty, quarter, cls, nclass, lane, slot, rot_ok, tx, ty, tz, lst,
-                                       th, th_t, tr, tw1);
+                                       th, th_t, tr, tw0, tw1);
                 if (++tx == a.ntx) {
                     tx = 0;
                     if (++ty == a.nty) {
