@@ -135,7 +135,10 @@ typedef enum {
     DOCK_TUNE_REGIONS = 1,        /* translation regions per rotation batch (0 = auto) */
     DOCK_TUNE_FORCE_FALLBACK = 2, /* 1 => every rotation takes the exact full-grid fallback (tests) */
     DOCK_TUNE_CAND_CAP = 3,       /* candidates kept per rotation before overflow fallback (>= 32) */
-    DOCK_TUNE_ENGINE = 4,         /* correlation engine: 0 auto (tcgen05 when eligible), 1 FP32 FFMA, 2 tcgen05 */
+    DOCK_TUNE_ENGINE = 4,         /* correlation engine: 0 auto (tcgen05 when eligible), 1 FP32 FFMA, 2 tcgen05,
+                                     3 FFT (cuFFT R2C/C2R + this library's channel multiply-accumulate and exact
+                                     greedy on the score grids; the paper's FFT method P:L156-163, kept as the
+                                     comparison point of the direct-vs-FFT crossover P:L485-502; never auto) */
     DOCK_TUNE_TC_VARIANT = 5,     /* tcgen05 kernel: 0 auto, 1 = resident receptor boxes (one channel group, P <= 4,
                                      128 translations x 4 rows per tile), 2 = receptor streamed one (channel group,
                                      z-plane) unit at a time (any P <= 32, m <= 8; 64 / 128 / 160 translations per
@@ -160,7 +163,7 @@ typedef struct {
     double l2_bytes;           /* device L2 size (cudaDevAttrL2CacheSize) */
     double corr_ms_last;       /* CUDA-event duration of the last k_corr launch (dock_probe_batch), -1 if none */
     int n_sms;                 /* multiprocessors of the context's device */
-    int engine_last;           /* engine of the last correlation: 1 FP32 FFMA, 2 tcgen05 bf16x3 */
+    int engine_last;           /* engine of the last correlation: 1 FP32 FFMA, 2 tcgen05 bf16x3, 3 FFT */
     int tc_available;          /* 1 if the tcgen05 engine is available for m_max */
     int tc_variant_last;       /* tcgen05 variant of the last correlation (1 or 2), 0 if FFMA */
     int tc_ksteps_last;        /* K-steps (K = 16 each) per translation row executed by the last tcgen05 launch */

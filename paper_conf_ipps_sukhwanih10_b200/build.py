@@ -12,7 +12,8 @@ CSRC = os.path.join(PKG, "csrc")
 LIB = os.path.join(PKG, "libdock.so")
 # dock.cu = host logic + small kernels; launch_*.cu = one correlation-kernel family each (compiled in
 # parallel, then linked into one shared library)
-SOURCES = [os.path.join(CSRC, "dock.cu")] + sorted(glob.glob(os.path.join(CSRC, "launch_*.cu")))
+SOURCES = [os.path.join(CSRC, "dock.cu")] + sorted(glob.glob(os.path.join(CSRC, "launch_*.cu"))) + \
+    [os.path.join(CSRC, "fft_engine.cu")]
 HEADERS = (sorted(glob.glob(os.path.join(CSRC, "*.cuh"))) + sorted(glob.glob(os.path.join(CSRC, "*.h"))) +
            [os.path.join(ROOT, "include", "dock.h")])
 
@@ -63,7 +64,7 @@ def build_native(force: bool = False, verbose: bool = False) -> str:
             raise RuntimeError(f"nvcc failed compiling {os.path.basename(src)}")
     tmp = LIB + tag
     res = subprocess.run([_nvcc(), "-gencode", "arch=compute_100a,code=sm_100a", "-shared", "-o", tmp, *objs,
-                          "-lcuda"], capture_output=True, text=True)
+                          "-lcuda", "-lcufft"], capture_output=True, text=True)
     if res.returncode != 0:
         sys.stderr.write(res.stdout + res.stderr)
         raise RuntimeError("nvcc failed linking libdock.so")

@@ -21,6 +21,7 @@
 #include "dock_kernels.cuh"
 #include "dock_tc.cuh"
 #include "dock_launch.h"
+#include "dock_fft.h"
 
 static_assert(sizeof(dock_pose) == 16, "dock_pose must be 16 bytes");
 static_assert(sizeof(dk::PoseOut) == sizeof(dock_pose), "kernel pose layout mismatch");
@@ -66,7 +67,8 @@ struct dock_ctx {
     float* d_ones = nullptr;   // [P] ones (unweighted voxel export)
     MPlan plan[DOCK_MAX_M + 1];
     // tcgen05 engine
-    int engine = 0;            // DOCK_TUNE_ENGINE: 0 auto, 1 FFMA, 2 tensor cores
+    int engine = 0;            // DOCK_TUNE_ENGINE: 0 auto, 1 FFMA, 2 tensor cores, 3 FFT (comparison engine)
+    DockFft* fft = nullptr;    // FFT engine state (receptor transform, plans, work buffers), created on first use
     int engine_last = 0;
     int tc_variant = 0;        // DOCK_TUNE_TC_VARIANT: 0 auto, 1 resident boxes (P <= 4), 2 streamed planes
     int tc_variant_last = 0;
@@ -662,6 +664,63 @@ dock_status pack_weights_tc(dock_ctx* ctx, int m, int v, int n_slots, const floa
     return DOCK_OK;
 }
 
+// FFT engine (engine 3): score grids of n slots [slot0, slot0 + n) (dock_fft.h).
+dock_status run_grid_fft(dock_ctx* ctx, int m, int slot0, int n, const float* Lw, float* grid)
+{
+    if (!ctx->fft && !(ctx->fft = dock_fft_create())) return fail(ctx, DOCK_E_OOM, "FFT engine state");
+    const dk::Geo& G = ctx->geo;
+    cudaError_t e = dock_fft_grids(ctx->fft, ctx->d_rec, G.Xp, G.Yp, G.Zp, ctx->nx, ctx->ny, ctx->nz, ctx->P, m, Lw,
+                                   slot0, n, grid, ctx->stream);
+    if (e != cudaSuccess) return fail(ctx, DOCK_E_CUDA, "FFT engine: %s", cudaGetErrorString(e));
+    ctx->kernels_last += 5;   // memset, scatter, R2C, multiply-accumulate, C2R
+    return DOCK_OK;
+}
+
+// FFT engine poses: score grids in chunks, then the exact greedy of the fallback path.
+dock_status run_fft_poses(dock_ctx* ctx, int m, int n_units, int64_t unit_begin, int n_rot, int k, int rho,
+                          void* poses)
+{
+    const int chunk = std::min(n_units, dock_fft_batch(ctx->nx, ctx->ny, ctx->nz, ctx->P));
+    const size_t ncell = (size_t)ctx->nx * ctx->ny * ctx->nz;
+    TRY(ensure(ctx, ctx->grid, sizeof(float) * ncell * chunk));
+    TRY(ensure(ctx, ctx->slots, sizeof(int) * n_units));
+    TRY(ensure(ctx, ctx->picks, sizeof(unsigned long long) * chunk * k));
+    TRY(ensure_pinned(ctx, sizeof(int) * n_units));
+    int* h = static_cast<int*>(ctx->h_stage);
+    CU(cudaStreamSynchronize(ctx->stream));
+    for (int i = 0; i < n_units; i++) h[i] = i;   // output slot of grid i
+    CU(cudaMemcpyAsync(ctx->slots.p, h, sizeof(int) * n_units, cudaMemcpyHostToDevice, ctx->stream));
+    for (int c0 = 0; c0 < n_units; c0 += chunk) {
+        const int n = std::min(chunk, n_units - c0);
+        TRY(run_grid_fft(ctx, m, c0, n, static_cast<const float*>(ctx->Lw.p), static_cast<float*>(ctx->grid.p)));
+        dk::GreedyArgs ga{};
+        ga.grid = static_cast<const float*>(ctx->grid.p);
+        ga.slots = static_cast<const int*>(ctx->slots.p) + c0;
+        ga.picks = static_cast<unsigned long long*>(ctx->picks.p);
+        ga.n = n;
+        ga.k = k;
+        ga.rho = rho;
+        ga.n_rot = n_rot;
+        ga.nx = ctx->nx;
+        ga.ny = ctx->ny;
+        ga.nz = ctx->nz;
+        ga.unit_begin = unit_begin;
+        ga.poses = poses;
+        dk::k_fill_u64<<<1, 256, 0, ctx->stream>>>(ga.picks, (size_t)n * k, dk::KEY_MAX);
+        CU(cudaGetLastError());
+        const int per_grid = std::max(1, std::min(256, 2 * ctx->n_sms / std::max(1, n)));
+        for (int j = 0; j < k; j++) {
+            ga.round = j;
+            dk::k_greedy_round<<<n * per_grid, 256, 0, ctx->stream>>>(ga);
+            CU(cudaGetLastError());
+        }
+        dk::k_greedy_emit<<<(n * k + 127) / 128, 128, 0, ctx->stream>>>(ga);
+        CU(cudaGetLastError());
+        ctx->kernels_last += k + 2;
+    }
+    return DOCK_OK;
+}
+
 // Score grids for n slots with the tensor-core engine (GRID epilogue).
 dock_status run_grid_tc(dock_ctx* ctx, int m, int n_slots, const float* Lw, float* grid)
 {
@@ -709,6 +768,7 @@ void dock_destroy(dock_ctx* ctx)
     for (DevBuf* b : bufs)
         if (b->p) cudaFree(b->p);
     if (ctx->d_trace) cudaFree(ctx->d_trace);
+    if (ctx->fft) dock_fft_destroy(ctx->fft);
     if (ctx->d_rec) cudaFree(ctx->d_rec);
     if (ctx->d_rec_tc) cudaFree(ctx->d_rec_tc);
     if (ctx->d_rec_pair) cudaFree(ctx->d_rec_pair);
@@ -889,7 +949,8 @@ dock_status dock_set_tuning(dock_ctx* ctx, int key, int64_t value)
             return DOCK_OK;
         case DOCK_TUNE_FORCE_FALLBACK: ctx->force_fallback = value ? 1 : 0; return DOCK_OK;
         case DOCK_TUNE_ENGINE:
-            if (value < 0 || value > 2) return fail(ctx, DOCK_E_INVALID_ARG, "engine must be 0 (auto), 1 (FFMA) or 2 (tcgen05)");
+            if (value < 0 || value > 3)
+                return fail(ctx, DOCK_E_INVALID_ARG, "engine must be 0 (auto), 1 (FFMA), 2 (tcgen05) or 3 (FFT)");
             ctx->engine = (int)value;
             return DOCK_OK;
         case DOCK_TUNE_TC_VARIANT:
@@ -1013,6 +1074,25 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
     // a1: voxelize (+ rotation / box validation)
     TRY(run_voxelize(ctx, m, n_units, unit_begin, nullptr, n_rot, d_xyz, d_coef, d_off, d_rot, ctx->d_w,
                      static_cast<float*>(ctx->Lw.p)));
+
+    if (ctx->engine == 3) {
+        // comparison engine: FFT score grids + exact greedy (no fused top-k, no fallback needed)
+        ctx->engine_last = 3;
+        ctx->tc_variant_last = 0;
+        CU(cudaEventRecord(ctx->ev_corr[0], ctx->stream));
+        TRY(run_fft_poses(ctx, m, n_units, unit_begin, n_rot, k, rho, d_poses));
+        CU(cudaEventRecord(ctx->ev_corr[1], ctx->stream));
+        ctx->ev_corr_valid = true;
+        ctx->fallback_last = 0;
+        CU(cudaMemcpyAsync(ctx->h_small, ctx->d_small, 16, cudaMemcpyDeviceToHost, ctx->stream));
+        CU(cudaStreamSynchronize(ctx->stream));
+        TRY(check_status_word(ctx));
+        if (!out_dev)
+            CU(cudaMemcpyAsync(out, d_poses, sizeof(dock_pose) * (size_t)n_units * k, cudaMemcpyDeviceToHost,
+                               ctx->stream));
+        CU(cudaStreamSynchronize(ctx->stream));
+        return DOCK_OK;
+    }
 
     // a2-a5: correlation + fused weighted score + on-chip top-k lists (no score grid in HBM)
     bool use_tc = false;
@@ -1151,8 +1231,10 @@ dock_status dock_score_grid(dock_ctx* ctx, const dock_probe_desc* probe, const d
     float* g_pt = per_term ? (pt_dev ? per_term : static_cast<float*>(ctx->grid.p) + (out_dev ? 0 : ncell)) : nullptr;
     CU(cudaMemsetAsync(ctx->d_small, 0, 4, ctx->stream));
     bool use_tc = false;
-    TRY(select_engine(ctx, m, &use_tc));
+    if (ctx->engine == 3) ctx->engine_last = 3;
+    else TRY(select_engine(ctx, m, &use_tc));
     auto grid_fn = [&](float* dst) -> dock_status {
+        if (ctx->engine == 3) return run_grid_fft(ctx, m, 0, 1, static_cast<const float*>(ctx->Lw.p), dst);
         return use_tc ? run_grid_tc(ctx, m, 1, static_cast<const float*>(ctx->Lw.p), dst)
                       : run_grid(ctx, m, 1, static_cast<const float*>(ctx->Lw.p), dst);
     };
