@@ -73,9 +73,11 @@ struct DockFft {
     float2* Lhat = nullptr;           // [B][P][nc]
     float2* Shat = nullptr;           // [B][nc]
     int cap = 0;                      // B the buffers hold
-    cufftHandle fwd = 0, inv = 0;     // batched R2C (B*P) and C2R (B) plans for batch `plan_n`
-    int plan_n = 0;
-    bool plans = false;
+    int m_last = 0;                   // ligand size of the last scatter (Lpad outside [0,m)^3 stays zero)
+    struct Plans {
+        cufftHandle fwd = 0, inv = 0;   // batched R2C (n*P) and C2R (n) plans
+        int n = 0;
+    } plans[2];                         // the full chunk and the tail chunk of a call
 };
 
 DockFft* dock_fft_create() { return new DockFft(); }
@@ -89,11 +91,13 @@ static void free_bufs(DockFft* f)
     f->Lhat = nullptr;
     f->Shat = nullptr;
     f->cap = 0;
-    if (f->plans) {
-        cufftDestroy(f->fwd);
-        cufftDestroy(f->inv);
-        f->plans = false;
-        f->plan_n = 0;
+    f->m_last = 0;
+    for (auto& pl : f->plans) {
+        if (pl.n) {
+            cufftDestroy(pl.fwd);
+            cufftDestroy(pl.inv);
+            pl.n = 0;
+        }
     }
 }
 
@@ -109,7 +113,7 @@ int dock_fft_batch(int nx, int ny, int nz, int P)
 {
     const double cells = double(nx) * ny * nz;
     const double per = cells * 4.0 * P + cells * 4.2 * P + cells * 4.2;   // Lpad + Lhat + Shat per grid
-    return (int)std::max(1.0, std::min(64.0, 2.0e9 / per));
+    return (int)std::max(1.0, std::min(64.0, 6.0e9 / per));
 }
 
 #define CK(x)                                         \
@@ -159,27 +163,35 @@ cudaError_t dock_fft_grids(DockFft* f, const float* rec, int Xp, int Yp, int Zp,
         CK(cudaMalloc(&f->Shat, sizeof(float2) * nc * n));
         f->cap = n;
     }
-    if (!f->plans || f->plan_n != n) {
-        if (f->plans) {
-            cufftDestroy(f->fwd);
-            cufftDestroy(f->inv);
-            f->plans = false;
+    // plans for this batch size: two cached (the full chunk and the tail of a call)
+    DockFft::Plans* pl = nullptr;
+    for (auto& c : f->plans)
+        if (c.n == n) pl = &c;
+    if (!pl) {
+        pl = f->plans[0].n == 0 ? &f->plans[0] : &f->plans[1];
+        if (pl->n) {
+            cufftDestroy(pl->fwd);
+            cufftDestroy(pl->inv);
+            pl->n = 0;
         }
-        FK(cufftPlanMany(&f->fwd, 3, dims, nullptr, 1, 0, nullptr, 1, 0, CUFFT_R2C, P * n));
-        FK(cufftPlanMany(&f->inv, 3, dims, nullptr, 1, 0, nullptr, 1, 0, CUFFT_C2R, n));
-        f->plans = true;
-        f->plan_n = n;
+        FK(cufftPlanMany(&pl->fwd, 3, dims, nullptr, 1, 0, nullptr, 1, 0, CUFFT_R2C, P * n));
+        FK(cufftPlanMany(&pl->inv, 3, dims, nullptr, 1, 0, nullptr, 1, 0, CUFFT_C2R, n));
+        pl->n = n;
     }
-    FK(cufftSetStream(f->fwd, st));
-    FK(cufftSetStream(f->inv, st));
-    CK(cudaMemsetAsync(f->Lpad, 0, sizeof(float) * cells * P * n, st));
+    FK(cufftSetStream(pl->fwd, st));
+    FK(cufftSetStream(pl->inv, st));
+    // the scatter only writes [0,m)^3 of every padded grid: zero the buffer only when m changes
+    if (m != f->m_last) {
+        CK(cudaMemsetAsync(f->Lpad, 0, sizeof(float) * cells * P * f->cap, st));
+        f->m_last = m;
+    }
     const int m3 = m * m * m;
     k_fft_scatter<<<std::max(1, std::min(1024, (n * P * m3 + 255) / 256)), 256, 0, st>>>(Lw, f->Lpad, slot0, n, P, m,
                                                                                       nx, ny, nz);
     CK(cudaGetLastError());
-    FK(cufftExecR2C(f->fwd, f->Lpad, reinterpret_cast<cufftComplex*>(f->Lhat)));
+    FK(cufftExecR2C(pl->fwd, f->Lpad, reinterpret_cast<cufftComplex*>(f->Lhat)));
     k_fft_mac<<<2048, 256, 0, st>>>(f->Rhat, f->Lhat, f->Shat, nc, n, P, 1.0f / static_cast<float>(cells));
     CK(cudaGetLastError());
-    FK(cufftExecC2R(f->inv, reinterpret_cast<cufftComplex*>(f->Shat), S));
+    FK(cufftExecC2R(pl->inv, reinterpret_cast<cufftComplex*>(f->Shat), S));
     return cudaGetLastError();
 }
