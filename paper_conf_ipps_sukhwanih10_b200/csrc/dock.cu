@@ -573,9 +573,10 @@ dock_status run_fallback(dock_ctx* ctx, int m, int nfb, int64_t unit_begin, int 
         ga.nz = ctx->nz;
         ga.unit_begin = unit_begin;
         ga.poses = poses;
+        ga.flag_bits = 1u;   // DOCK_POSE_FALLBACK
         dk::k_fill_u64<<<1, 256, 0, ctx->stream>>>(ga.picks, (size_t)n * k, dk::KEY_MAX);
         CU(cudaGetLastError());
-        const int per_grid = std::max(1, std::min(256, 2 * ctx->n_sms / std::max(1, n)));
+        const int per_grid = std::max(8, std::min(512, 16 * ctx->n_sms / std::max(1, n)));
         for (int j = 0; j < k; j++) {
             ga.round = j;
             dk::k_greedy_round<<<n * per_grid, 256, 0, ctx->stream>>>(ga);
@@ -706,9 +707,10 @@ dock_status run_fft_poses(dock_ctx* ctx, int m, int n_units, int64_t unit_begin,
         ga.nz = ctx->nz;
         ga.unit_begin = unit_begin;
         ga.poses = poses;
+        ga.flag_bits = 0u;
         dk::k_fill_u64<<<1, 256, 0, ctx->stream>>>(ga.picks, (size_t)n * k, dk::KEY_MAX);
         CU(cudaGetLastError());
-        const int per_grid = std::max(1, std::min(256, 2 * ctx->n_sms / std::max(1, n)));
+        const int per_grid = std::max(8, std::min(512, 16 * ctx->n_sms / std::max(1, n)));
         for (int j = 0; j < k; j++) {
             ga.round = j;
             dk::k_greedy_round<<<n * per_grid, 256, 0, ctx->stream>>>(ga);

@@ -643,6 +643,7 @@ struct GreedyArgs {
     int nx, ny, nz;
     long long unit_begin;
     void* poses;
+    unsigned flag_bits;         // pose flags of these picks: DOCK_POSE_FALLBACK (1) on the fallback path, 0 (FFT engine)
 };
 
 // One round j of the paper's best-then-exclude loop over full score grids,
@@ -663,13 +664,23 @@ __global__ void k_greedy_round(GreedyArgs a)
     if (j > 0 && pk[j - 1] == KEY_MAX) return;   // fewer than j picks possible
     unsigned long long best = KEY_MAX;
     const uint32_t stride = static_cast<uint32_t>(ctas_per_grid) * blockDim.x;
-    for (uint32_t t = part * blockDim.x + threadIdx.x; t < ncell; t += stride) {
-        const unsigned long long key = make_key(S[t], t);
-        if (key >= best) continue;
+    auto consider = [&](uint32_t t, float sv) {
+        const unsigned long long key = make_key(sv, t);
+        if (key >= best) return;
         bool ok = true;
         for (int q = 0; q < j; q++) ok = ok && (cheb_cyc(t, prev[q], a.nx, a.ny, a.nz) > a.rho);
         if (ok) best = key;
+    };
+    // four independent loads in flight per thread (the scan is bandwidth-, not compute-bound)
+    uint32_t t = part * blockDim.x + threadIdx.x;
+    for (; t + 3 * stride < ncell; t += 4 * stride) {
+        const float s0 = S[t], s1 = S[t + stride], s2 = S[t + 2 * stride], s3 = S[t + 3 * stride];
+        consider(t, s0);
+        consider(t + stride, s1);
+        consider(t + 2 * stride, s2);
+        consider(t + 3 * stride, s3);
     }
+    for (; t < ncell; t += stride) consider(t, S[t]);
     best = warp_min_u64(best);
     if ((threadIdx.x & 31) == 0 && best != KEY_MAX) atomicMin(&pk[j], best);
 }
@@ -690,11 +701,11 @@ __global__ void k_greedy_emit(GreedyArgs a)
     if (key != KEY_MAX) {
         po.t_lin = static_cast<int32_t>(key & 0xffffffffu);
         po.score = unord_f32(static_cast<uint32_t>(key >> 32));
-        po.flags = 1u;
+        po.flags = a.flag_bits;
     } else {
         po.t_lin = -1;
         po.score = __int_as_float(0x7fc00000);
-        po.flags = 3u;
+        po.flags = a.flag_bits | 2u;
     }
     reinterpret_cast<PoseOut*>(a.poses)[static_cast<size_t>(slot) * a.k + j] = po;
 }

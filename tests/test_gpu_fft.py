@@ -70,6 +70,7 @@ def test_fft_poses(D, orc, rho, k):
         L = orc.voxelize(pr.xyz, pr.coef, m, rot[r], H)
         S, A = orc.score_grid(R, L, w)
         assert (poses[u]["rot"] == r).all()
+        assert (poses[u]["flags"] == 0).all()   # exact greedy on full grids: no fallback flag
         validate_unit(S, A, poses[u]["t_lin"], poses[u]["score"], k, rho)
 
 
