@@ -386,7 +386,11 @@ def run_ours(args):
                      "fallback_rotations": fallbacks, "timing": "CUDA events on the context stream"})
         line = {"metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world, "steps": args.steps,
                 "warmup": args.warmup, "ms_per_step": ms_step, "higher_is_better": True, "scaling": "strong",
-                "vs_baseline": None, "dtype": "f32", "data": "synthetic", "config": desc,
+                "vs_baseline": None,
+                # tcgen05: bf16 products of hi/lo splits (bf16x3) accumulated in f32 (scores within 1e-4*A of
+                # FP64, reading Q16); FFMA: plain f32
+                "dtype": "bf16x3 split, f32 accumulate" if info["engine_last"] == 2 else "f32",
+                "data": "synthetic", "config": desc,
                 "e2e": e2e, "gpu_launches": launches, "roofline": roof, "cpu_baseline": cpu, "clocks": clocks,
                 "engine": roof["engine"], "alt_engine": alt}
         print(json.dumps(line), flush=True)
