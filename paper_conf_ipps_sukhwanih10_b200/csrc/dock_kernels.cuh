@@ -575,8 +575,9 @@ struct PoseOut {
 // One warp per rotation.  Greedy over the candidate set W: k times take the minimum key
 // that is farther than rho (cyclic Chebyshev) from every earlier pick.
 // W contains every warp list's keys <= the final pruning bound T >= key(g_k); the result
-// equals the exact full-grid greedy when every warp list's 32nd key exceeds the last pick
-// (mu > key(c_k)); otherwise, or on candidate overflow, the rotation is flagged for the
+// equals the exact full-grid greedy when no list's last key is below the last pick
+// (mu >= key(c_k): keys are unique, so a key <= a full list's last key is in that list);
+// otherwise, or on candidate overflow, the rotation is flagged for the
 // exact fallback (DESIGN.md §Top-k exactness).
 #ifndef DOCK_LAUNCHER_TU   // defined once, in dock.cu
 __global__ void k_merge(MergeArgs a)
@@ -609,7 +610,7 @@ __global__ void k_merge(MergeArgs a)
         np++;
     }
     const bool sound = !a.force_fallback && n_all <= static_cast<unsigned int>(a.cap) && np == a.k &&
-                       a.mu[slot] > picks[a.k - 1];
+                       a.mu[slot] >= picks[a.k - 1];   // keys are unique: a key <= a list's last key is in it
     const long long unit = a.unit_begin + slot;
     PoseOut* out = reinterpret_cast<PoseOut*>(a.poses) + static_cast<size_t>(slot) * a.k;
     for (int j = lane; j < a.k; j += 32) {
