@@ -39,7 +39,7 @@ constexpr int NT = 128;         // translations per row (MMA N)
 #define DOCK_TC_STAIR 3
 #endif
 constexpr int NEPI_MAX = DOCK_TC_NEPI_MAX;   // epilogue warps: a.nepi in {4, 8} (1 or 2 per TMEM lane quarter; 8 measured best: 168 registers per thread, 2 row classes)
-constexpr int NTHREADS = (2 + NEPI_MAX) * 32;   // launch bound; the launch uses (2 + a.nepi) * 32 threads
+constexpr int NTHREADS = (3 + NEPI_MAX) * 32;   // launch bound; both variants launch (3 + a.nepi) * 32 threads
 constexpr int WSTAGES = 16;     // max weight ring depth (runtime a.wstages <= 16; 16 x 4 KB covers the L2 latency)
 constexpr int WCHUNK = 2 * ROT * 16;   // bytes of one K-step of A (2 K-chunks x 128 rotations x 16 B)
 constexpr int KSTEPS = 4;       // K-steps of A per ring stage (one elected issue block of KSTEPS*Q MMAs)
@@ -398,73 +398,55 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
     long long tw0 = 0, tw1 = 0, tw2 = 0, tstart = tr ? clock64() : 0;   // per-role trace accumulators
     if (n_tiles > 0) {
         if (warp == 0) {
-            // ------------------------------------------------ TMA producer (warp-converged, one elected lane)
+            // ------------------------------------------------ weight producer (one thread): the whole A
+            // stream in stage order; it never waits on a receptor buffer (warp 2 + nepi loads those)
+            if (elect_one()) {
+                const unsigned char* wsrc = a.W + static_cast<size_t>(block) * NSTEPS * WCHUNK;
+                int ws = 0, wph = 0, wuse = 0;
+                for (int ti = 0; ti < n_tiles; ti++) {
+                    for (int s = 0; s < NSTEPS; s += KS) {
+                        if (wuse >= a.wstages) twait(&w_empty[ws], wph ^ 1, tr, tw0);
+                        dk::mbar_arrive_expect_tx(&w_full[ws], STAGE);
+                        dk::bulk_load(w_smem + static_cast<size_t>(ws) * STAGE,
+                                      wsrc + static_cast<size_t>(s) * WCHUNK, STAGE, &w_full[ws]);
+                        wuse++;
+                        if (++ws == a.wstages) {
+                            ws = 0;
+                            wph ^= 1;
+                        }
+                    }
+                }
+                if (tr) {
+                    atomicAdd(&a.trace[TR_PROD_TOTAL], static_cast<unsigned long long>(clock64() - tstart));
+                    atomicAdd(&a.trace[TR_PROD_WEMPTY], static_cast<unsigned long long>(tw0));
+                    atomicAdd(&a.trace[TR_CTAS], 1ull);
+                    atomicAdd(&a.trace[TR_TILES], static_cast<unsigned long long>(n_tiles));
+                }
+            }
+            __syncwarp();
+        } else if (warp == 2 + a.nepi) {
+            // ------------------------------------------------ receptor producer (one thread): main box of
+            // tile t as soon as pass 1 of t-1 released it, pair box as soon as pass 2 of t-1 did
             if (elect_one()) {
                 dk::prefetch_tmap(&tmap);
                 dk::prefetch_tmap(&tmap_pair);
-            }
-            const unsigned char* wsrc = a.W + static_cast<size_t>(block) * NSTEPS * WCHUNK;
-            int ws = 0, wph = 0;                  // weight ring slot / phase
-            int wuse = 0;
-            auto stream_weights = [&](int s) {
-                if (wuse >= a.wstages) twait(&w_empty[ws], wph ^ 1, tr, tw0);
-                if (elect_one()) {
-                    dk::mbar_arrive_expect_tx(&w_full[ws], STAGE);
-                    dk::bulk_load(w_smem + static_cast<size_t>(ws) * STAGE, wsrc + static_cast<size_t>(s) * WCHUNK,
-                                  STAGE, &w_full[ws]);
+                int tx = tile_begin % a.ntx, ty = (tile_begin / a.ntx) % a.nty, tz = tile_begin / (a.ntx * a.nty);
+                for (int ti = 0; ti < n_tiles; ti++) {
+                    for (int which = 0; which < 2; which++) {
+                        if (ti > 0) twait(&rec_empty[which], (ti - 1) & 1, tr, tw1);
+                        dk::mbar_arrive_expect_tx(&rec_full[which], a.box_bytes);
+                        tma_load_5d(rec_smem + which * a.rec_stage_bytes, which ? &tmap_pair : &tmap, 0, tx * NT,
+                                    ty * Q, tz, 0, &rec_full[which]);
+                    }
+                    if (++tx == a.ntx) {
+                        tx = 0;
+                        if (++ty == a.nty) {
+                            ty = 0;
+                            tz++;
+                        }
+                    }
                 }
-                __syncwarp();
-                wuse++;
-                if (++ws == a.wstages) {
-                    ws = 0;
-                    wph ^= 1;
-                }
-            };
-            // Receptor boxes are issued as soon as their buffer frees: the producer polls the release
-            // barriers between weight stages (main(t+1) needs pass 1 of t done, pair(t+1) pass 2 of t),
-            // and blocks only right before the first stage that needs a box.
-            int pm = 0, pp = 0;   // next main / pair box (tile index) to load
-            auto issue_box = [&](int which, int t) {
-                const int tile = tile_begin + t;
-                const int tx = tile % a.ntx, ty = (tile / a.ntx) % a.nty, tz = tile / (a.ntx * a.nty);
-                if (elect_one()) {
-                    dk::mbar_arrive_expect_tx(&rec_full[which], a.box_bytes);
-                    tma_load_5d(rec_smem + which * a.rec_stage_bytes, which ? &tmap_pair : &tmap, 0, tx * NT, ty * Q,
-                                tz, 0, &rec_full[which]);
-                }
-                __syncwarp();
-            };
-            auto poll = [&](int ti) {
-                if (pm < n_tiles && pm <= ti + 1 && (pm == 0 || dk::mbar_test(&rec_empty[0], (pm - 1) & 1)))
-                    issue_box(0, pm++);
-                if (pp < n_tiles && pp <= ti + 1 && (pp == 0 || dk::mbar_test(&rec_empty[1], (pp - 1) & 1)))
-                    issue_box(1, pp++);
-            };
-            auto ensure = [&](int which, int t) {
-                int& nx = which ? pp : pm;
-                if (nx == t) {
-                    if (t > 0) twait(&rec_empty[which], (t - 1) & 1, tr, tw1);
-                    issue_box(which, nx++);
-                }
-            };
-            for (int ti = 0; ti < n_tiles; ti++) {
-                ensure(0, ti);
-                for (int s = 0; s < S1P; s += KS) {
-                    poll(ti);
-                    stream_weights(s);
-                }
-                ensure(1, ti);
-                for (int s = S1P; s < NSTEPS; s += KS) {
-                    poll(ti);
-                    stream_weights(s);
-                }
-            }
-            if (tr && elect_one()) {
-                atomicAdd(&a.trace[TR_PROD_TOTAL], static_cast<unsigned long long>(clock64() - tstart));
-                atomicAdd(&a.trace[TR_PROD_WEMPTY], static_cast<unsigned long long>(tw0));
-                atomicAdd(&a.trace[TR_PROD_REMPTY], static_cast<unsigned long long>(tw1));
-                atomicAdd(&a.trace[TR_CTAS], 1ull);
-                atomicAdd(&a.trace[TR_TILES], static_cast<unsigned long long>(n_tiles));
+                if (tr) atomicAdd(&a.trace[TR_PROD_REMPTY], static_cast<unsigned long long>(tw1));
             }
             __syncwarp();
         } else if (warp == 1) {
@@ -739,13 +721,38 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tcs(const __grid_constant_
     long long tw0 = 0, tw1 = 0, tw2 = 0, tstart = tr ? clock64() : 0;
     if (n_tiles > 0) {
         if (warp == 0) {
-            // ------------------------------------------------ TMA producer (one thread), in unit order:
-            // the unit's two planes into the next receptor slot, then its weight stages into the ring
+            // ------------------------------------------------ weight producer (one thread): the A stream in
+            // unit order; receptor planes are loaded by warp 2 + nepi, so this thread never waits on a slot
+            if (elect_one()) {
+                const unsigned char* wsrc = a.W + static_cast<size_t>(block) * a.nsteps * WCHUNK;
+                int ws = 0, wph = 0, wuse = 0;
+                for (int ti = 0; ti < n_tiles; ti++) {
+                    for (int s = 0; s < a.nsteps; s += KS) {
+                        if (wuse >= a.wstages) twait(&w_empty[ws], wph ^ 1, tr, tw0);
+                        dk::mbar_arrive_expect_tx(&w_full[ws], STAGE);
+                        dk::bulk_load(w_smem + static_cast<size_t>(ws) * STAGE, wsrc + static_cast<size_t>(s) * WCHUNK,
+                                      STAGE, &w_full[ws]);
+                        wuse++;
+                        if (++ws == a.wstages) {
+                            ws = 0;
+                            wph ^= 1;
+                        }
+                    }
+                }
+                if (tr) {
+                    atomicAdd(&a.trace[TR_PROD_TOTAL], static_cast<unsigned long long>(clock64() - tstart));
+                    atomicAdd(&a.trace[TR_PROD_WEMPTY], static_cast<unsigned long long>(tw0));
+                    atomicAdd(&a.trace[TR_CTAS], 1ull);
+                    atomicAdd(&a.trace[TR_TILES], static_cast<unsigned long long>(n_tiles));
+                }
+            }
+            __syncwarp();
+        } else if (warp == 2 + a.nepi) {
+            // ------------------------------------------------ receptor producer (one thread): each unit's two
+            // z-planes into the next ring slot as soon as the MMAs of the unit NR earlier released it
             if (elect_one()) {
                 dk::prefetch_tmap(&tmap);
                 dk::prefetch_tmap(&tmap_pair);
-                const unsigned char* wsrc = a.W + static_cast<size_t>(block) * a.nsteps * WCHUNK;
-                int ws = 0, wph = 0, wuse = 0;
                 int rs = 0, rph = 0, ruse = 0;
                 int tx = tile_begin % a.ntx, ty = (tile_begin / a.ntx) % a.nty, tz = tile_begin / (a.ntx * a.nty);
                 for (int ti = 0; ti < n_tiles; ti++) {
@@ -761,18 +768,6 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tcs(const __grid_constant_
                             rs = 0;
                             rph ^= 1;
                         }
-                        const unsigned char* wu = wsrc + static_cast<size_t>(u) * KUP * WCHUNK;
-                        for (int st = 0; st < NSU; st++) {
-                            if (wuse >= a.wstages) twait(&w_empty[ws], wph ^ 1, tr, tw0);
-                            dk::mbar_arrive_expect_tx(&w_full[ws], STAGE);
-                            dk::bulk_load(w_smem + static_cast<size_t>(ws) * STAGE,
-                                          wu + static_cast<size_t>(st) * STAGE, STAGE, &w_full[ws]);
-                            wuse++;
-                            if (++ws == a.wstages) {
-                                ws = 0;
-                                wph ^= 1;
-                            }
-                        }
                     }
                     if (++tx == a.ntx) {
                         tx = 0;
@@ -782,13 +777,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tcs(const __grid_constant_
                         }
                     }
                 }
-                if (tr) {
-                    atomicAdd(&a.trace[TR_PROD_TOTAL], static_cast<unsigned long long>(clock64() - tstart));
-                    atomicAdd(&a.trace[TR_PROD_WEMPTY], static_cast<unsigned long long>(tw0));
-                    atomicAdd(&a.trace[TR_PROD_REMPTY], static_cast<unsigned long long>(tw1));
-                    atomicAdd(&a.trace[TR_CTAS], 1ull);
-                    atomicAdd(&a.trace[TR_TILES], static_cast<unsigned long long>(n_tiles));
-                }
+                if (tr) atomicAdd(&a.trace[TR_PROD_REMPTY], static_cast<unsigned long long>(tw1));
             }
             __syncwarp();
         } else if (warp == 1) {

@@ -9,7 +9,7 @@ static cudaError_t launch_t(const CUtensorMap& tmap, const CUtensorMap& tmap_pai
     auto kern = tc::k_corr_tc<M, GRID>;
     cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
     if (e != cudaSuccess) return e;
-    kern<<<nblocks, (2 + a.nepi) * 32, smem, st>>>(tmap, tmap_pair, a);
+    kern<<<nblocks, (3 + a.nepi) * 32, smem, st>>>(tmap, tmap_pair, a);   // + receptor producer warp
     return cudaGetLastError();
 }
 
