@@ -357,3 +357,36 @@ def test_large_config_sampled(D, orc, engine):
     rot = g.rotations(256, seed=3001)
     _, info, _ = _dock_and_validate(D, orc, R, w, probes, rot, c.k, 1, units=[0, 173], engine=engine)
     assert info["fallback_last"] <= 4 and _engine_id(info) == engine
+
+
+# ----------------------------------------------------------------------------- maximum / degenerate sizes
+
+
+@pytest.mark.parametrize("engine", ENGINES)
+@pytest.mark.parametrize("rho", [0, 1])
+def test_max_terms_probe_and_k(D, orc, engine, rho):
+    """DOCK_MAX_TERMS = 32 channels (8 tcgen05 channel groups), the largest probe grid m = 8 and
+    DOCK_MAX_K = 32 poses per rotation, on a ragged grid; poses validated tie-aware, score grids
+    within 1e-4 * A."""
+    P, m, k = D.DOCK_MAX_TERMS, D.DOCK_MAX_M, D.DOCK_MAX_K
+    R = g.receptor("uniform", (48, 20, 17), P)
+    w = g.weights(P)
+    probes = g.probes(1, m, P)
+    rot = g.rotations(5, with_cube_group=False)
+    poses, info, _ = _dock_and_validate(D, orc, R, w, probes, rot, k, rho, engine=engine)
+    assert _engine_id(info) == (1 if engine == 1 else 3)   # 8 channel groups: tcgen05 variant 2
+    ctx = _ctx(D, R, w, m, engine)
+    S_g = D.dock_score_grid(ctx, probes[0], rot[1])
+    ctx.close()
+    S_o, A_o = _oracle_SA(orc, R, w, probes[0], rot[1])
+    assert (np.abs(S_g.astype(np.float64) - S_o) <= 1e-4 * A_o + 1e-12).all()
+
+
+def test_empty_unit_range(D):
+    """An empty shard (unit_begin == unit_end) is a no-op, not an error."""
+    P, m = 4, 4
+    R = g.receptor_ftmap_like((32, 32, 32), P)
+    ctx = D.dock_init(R, g.weights(P), H, m_max=m)
+    out = D.dock_probe_batch(ctx, g.probes(1, m, P), g.rotations(4), unit_begin=2, unit_end=2, k=4, rho=1)
+    assert len(out) == 0
+    ctx.close()
