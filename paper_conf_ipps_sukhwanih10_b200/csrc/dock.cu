@@ -40,7 +40,8 @@ struct TcPlan {                // per-(variant, probe size) plan of the tcgen05 
     CUtensorMap tmap, tmap_pair;   // (hi,lo) receptor copy and PAIR copy (Rhi(x), Rhi(x+1))
     int ntt = 0, q = 0, ntx = 0, nty = 0, ntiles = 0;   // translations per row, rows per tile, tile counts
     int S1 = 0, S1p = 0, S2 = 0, S2p = 0;                // variant 1: pass-1 / pass-2 K-steps (real, padded)
-    int box_bytes = 0, rec_stage_bytes = 0, n_rec_stages = 0, smem = 0, nsteps = 0, wstages = 0;
+    int box_bytes = 0, box_bytes_pair = 0, rec_stage_bytes = 0, n_rec_stages = 0, smem = 0, nsteps = 0, wstages = 0;
+    int TXBP = 0;              // variant 1: x extent of the pair box (the main box uses TXB of make_tc_plan)
 };
 
 struct MPlan {                 // per-probe-size launch plan
@@ -263,18 +264,22 @@ dock_status make_tc_plan(dock_ctx* ctx, int m, int v)
     TcPlan& pl = ctx->tcplan[v][m];
     if (pl.ok || !ctx->d_rec_tc || !ctx->d_rec_pair) return DOCK_OK;
     const int KS = tc::KSTEPS;
-    const int budget = kSmemLimit - 2048;   // static shared memory (barriers) and slack
+    const int budget = kSmemLimit - 512;    // static shared memory (barriers: < 400 B)
     const int stage = KS * tc::WCHUNK;
     int TXB = 0, TYB = 0, TZB = 0;
+    int rec_bytes = 0;   // shared memory before the weight ring
     if (v == 1) {
         if (ctx->tc_Gch != 1) return DOCK_OK;   // one channel group only
         pl.ntt = tc::NT;
         pl.q = 4;
-        TXB = tc::pair_txb(m, pl.ntt);
+        TXB = tc::main_box_txb(m);
+        pl.TXBP = tc::pair_box_txb(m);
         TYB = pl.q + m - 1;
         TZB = m;
         pl.box_bytes = 16 * TXB * TYB * TZB;
-        pl.rec_stage_bytes = round_up(pl.box_bytes, 1024);
+        pl.box_bytes_pair = 16 * pl.TXBP * TYB * TZB;
+        pl.rec_stage_bytes = round_up(pl.box_bytes, 128);   // offset of the pair box
+        rec_bytes = pl.rec_stage_bytes + round_up(pl.box_bytes_pair, 128);
         pl.n_rec_stages = 2;   // main box + pair box
         const int MXP = (m + 1) / 2, MXQ = (m + 3) / 4;
         pl.S1 = m * m * MXP;
@@ -282,7 +287,7 @@ dock_status make_tc_plan(dock_ctx* ctx, int m, int v)
         pl.S2 = m * m * MXQ;
         pl.S2p = round_up(pl.S2, KS);
         pl.nsteps = pl.S1p + pl.S2p;
-        if (2 * pl.rec_stage_bytes + 3 * stage > budget) return DOCK_OK;   // not eligible for this m
+        if (rec_bytes + 3 * stage > budget) return DOCK_OK;   // not eligible for this m
     } else {
         pl.ntt = ctx->tcs_ntt;
         pl.q = tcs_q(pl.ntt);
@@ -293,25 +298,26 @@ dock_status make_tc_plan(dock_ctx* ctx, int m, int v)
         pl.rec_stage_bytes = round_up(2 * (int)tc::stream_plane_stride(m, pl.ntt, pl.q), 1024);
         pl.n_rec_stages = 3 * pl.rec_stage_bytes + 6 * stage <= budget ? 3 : 2;
         if (pl.n_rec_stages * pl.rec_stage_bytes + 3 * stage > budget) return DOCK_OK;
+        rec_bytes = pl.n_rec_stages * pl.rec_stage_bytes;
         pl.nsteps = ctx->tc_Gch * m * tc::unit_ksteps_padded(m);
     }
-    if (TXB > 256 || TYB > 256) return DOCK_OK;   // TMA box limit
+    if (TXB > 256 || TYB > 256 || pl.TXBP > 256) return DOCK_OK;   // TMA box limit
     pl.ntx = (ctx->nx + pl.ntt - 1) / pl.ntt;
     pl.nty = (ctx->ny + pl.q - 1) / pl.q;
     pl.ntiles = pl.ntx * pl.nty * ctx->nz;
-    if ((pl.ntx - 1) * pl.ntt + TXB > ctx->tc_Xp || pl.nty * pl.q + m - 1 > ctx->tc_Yp)
+    if ((pl.ntx - 1) * pl.ntt + std::max(TXB, pl.TXBP) > ctx->tc_Xp || pl.nty * pl.q + m - 1 > ctx->tc_Yp)
         return fail(ctx, DOCK_E_CUDA, "tcgen05 receptor padding too small");
-    pl.wstages = std::min(tc::WSTAGES, (budget - pl.n_rec_stages * pl.rec_stage_bytes) / stage);
+    pl.wstages = std::min(tc::WSTAGES, (budget - rec_bytes) / stage);
     // >= 116 KB keeps one CTA per SM: every CTA allocates all 512 TMEM columns
-    pl.smem = std::max(pl.n_rec_stages * pl.rec_stage_bytes + pl.wstages * stage, 116 * 1024);
+    pl.smem = std::max(rec_bytes + pl.wstages * stage, 116 * 1024);
     auto fn = encode_fn();
     if (!fn) return fail(ctx, DOCK_E_CUDA, "cuTensorMapEncodeTiled unavailable");
     const cuuint64_t X = ctx->tc_Xp, Y = ctx->tc_Yp, Z = ctx->tc_Zp;
     cuuint64_t dims[5] = {8, X, Y, Z, (cuuint64_t)ctx->tc_Gch};
     cuuint64_t strides[4] = {16, X * 16, X * Y * 16, X * Y * Z * 16};
-    cuuint32_t box[5] = {8, (cuuint32_t)TXB, (cuuint32_t)TYB, (cuuint32_t)TZB, 1};
     cuuint32_t es[5] = {1, 1, 1, 1, 1};
     for (int which = 0; which < 2; which++) {
+        cuuint32_t box[5] = {8, (cuuint32_t)(which && v == 1 ? pl.TXBP : TXB), (cuuint32_t)TYB, (cuuint32_t)TZB, 1};
         CUresult r = fn(which ? &pl.tmap_pair : &pl.tmap, CU_TENSOR_MAP_DATA_TYPE_BFLOAT16, 5,
                         which ? (void*)ctx->d_rec_pair : (void*)ctx->d_rec_tc, dims, strides, box, es,
                         CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_L2_256B,
@@ -607,6 +613,7 @@ tc::TcArgs tc_args(dock_ctx* ctx, int m, int v, int n_slots, int G, const unsign
     a.nsteps = tp.nsteps;
     a.W = W;
     a.box_bytes = tp.box_bytes;
+    a.box_bytes_pair = tp.box_bytes_pair;
     a.rec_stage_bytes = tp.rec_stage_bytes;
     a.n_rec_stages = tp.n_rec_stages;
     a.wstages = tp.wstages;

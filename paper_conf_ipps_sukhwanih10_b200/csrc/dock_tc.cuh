@@ -52,7 +52,8 @@ struct TcArgs {
     int n_slots, G, tiles_per_region;
     int nsteps;                 // K-steps of A per tile (all passes / units, padded to whole ring stages)
     const unsigned char* W;     // [block][step][WCHUNK]
-    int box_bytes;              // bytes of one receptor TMA box (variant 1: whole box; variant 2: one z-plane)
+    int box_bytes;              // bytes of one receptor TMA box (variant 1: the main box; variant 2: one z-plane)
+    int box_bytes_pair;         // variant 1: bytes of the pair box
     int rec_stage_bytes;        // variant 1: offset of the pair box; variant 2: one receptor ring slot (unit)
     int n_rec_stages;           // variant 2: receptor ring depth (units)
     int wstages;                // weight ring depth (3..WSTAGES)
@@ -313,6 +314,10 @@ __host__ __device__ constexpr int pair_txb(int m, int ntt = NT)
     return (ntt + (m + 1) / 2 * 2 - 1) > (4 * ((m + 3) / 4) + ntt - 2) ? (ntt + (m + 1) / 2 * 2 - 1)
                                                                        : (4 * ((m + 3) / 4) + ntt - 2);
 }
+// Variant 1 sizes each box to what its pass reads: main (hi,lo) box x extent NT + 2*MXP - 1, pair box
+// NT + 4*MXQ - 2 (slot x already holds voxel x + 1) -- at m = 4 the 448 B saved let a 7th weight stage fit.
+__host__ __device__ constexpr int main_box_txb(int m) { return NT + (m + 1) / 2 * 2 - 1; }
+__host__ __device__ constexpr int pair_box_txb(int m) { return NT + 4 * ((m + 3) / 4) - 2; }
 // Byte offset of K-step s inside the PAIR pass-1 box ((hi,lo) voxels, 2 per K-step) and pass-2 box
 // ((hi(x),hi(x+1)) slots, 4 voxels per K-step); padding steps (zero weights) re-read the last real
 // step's voxels.
@@ -348,10 +353,12 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
     constexpr int S1 = M * M * MXP, S1P = (S1 + KS - 1) / KS * KS;
     constexpr int S2 = M * M * MXQ, S2P = (S2 + KS - 1) / KS * KS;
     constexpr int NSTEPS = S1P + S2P;
-    constexpr uint32_t ROW16 = static_cast<uint32_t>(pair_txb(M)) * 16u;
+    constexpr uint32_t ROW16 = static_cast<uint32_t>(main_box_txb(M)) * 16u;    // main box row pitch
     constexpr uint32_t ROWTY = static_cast<uint32_t>(Q + M - 1) * ROW16;
+    constexpr uint32_t ROW16P = static_cast<uint32_t>(pair_box_txb(M)) * 16u;   // pair box row pitch
+    constexpr uint32_t ROWTYP = static_cast<uint32_t>(Q + M - 1) * ROW16P;
     static_assert(Q * NT <= 512, "TMEM has 512 columns");
-    extern __shared__ __align__(1024) unsigned char smem[];
+    extern __shared__ __align__(128) unsigned char smem[];   // TMA destinations: 128 B; no-swizzle UMMA operands: 16 B
     __shared__ uint64_t bars[2 * 2 + 2 * WSTAGES + 2 * Q];
     __shared__ uint32_t tmem_base_s;
     uint64_t* rec_full = bars;
@@ -366,8 +373,8 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
     const int tile_begin = region * a.tiles_per_region;
     const int tile_end = min(a.ntiles, tile_begin + a.tiles_per_region);
     const int n_tiles = tile_end - tile_begin;
-    unsigned char* rec_smem = smem;   // [main box | pair box], a.rec_stage_bytes each
-    unsigned char* w_smem = smem + 2 * a.rec_stage_bytes;
+    unsigned char* rec_smem = smem;   // [main box | pair box at a.rec_stage_bytes]
+    unsigned char* w_smem = smem + a.rec_stage_bytes + ((a.box_bytes_pair + 127) & ~127);
 
     if (threadIdx.x == 0) {
         for (int i = 0; i < 2; i++) {
@@ -434,7 +441,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                 for (int ti = 0; ti < n_tiles; ti++) {
                     for (int which = 0; which < 2; which++) {
                         if (ti > 0) twait(&rec_empty[which], (ti - 1) & 1, tr, tw1);
-                        dk::mbar_arrive_expect_tx(&rec_full[which], a.box_bytes);
+                        dk::mbar_arrive_expect_tx(&rec_full[which], which ? a.box_bytes_pair : a.box_bytes);
                         tma_load_5d(rec_smem + which * a.rec_stage_bytes, which ? &tmap_pair : &tmap, 0, tx * NT,
                                     ty * Q, tz, 0, &rec_full[which]);
                     }
@@ -547,7 +554,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
 #pragma unroll
                             for (int q = 0; q < Q; q++)
                                 umma_bf16(tmem + q * NT, da0 + ((ks * WCHUNK) >> 4),
-                                          dP0 + ((pair_off2(M, st * KS + ks, ROW16, ROWTY) + q * ROW16) >> 4), idesc,
+                                          dP0 + ((pair_off2(M, st * KS + ks, ROW16P, ROWTYP) + q * ROW16P) >> 4), idesc,
                                           1u);
                         umma_commit(&w_empty[ws]);
                         advance(1);
@@ -568,7 +575,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
 #pragma unroll
                             for (int ks = 0; ks < KS; ks++)
                                 umma_bf16(tmem + q * NT, da0 + ((ks * WCHUNK) >> 4),
-                                          dP0 + ((pair_off2(M, st * KS + ks, ROW16, ROWTY) + q * ROW16) >> 4), idesc,
+                                          dP0 + ((pair_off2(M, st * KS + ks, ROW16P, ROWTYP) + q * ROW16P) >> 4), idesc,
                                           1u);
                         }
                         umma_commit(&tm_full[q]);
@@ -674,7 +681,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tcs(const __grid_constant_
     constexpr int NRMAX = 4;
     static_assert(Q * NTT <= 512, "TMEM has 512 columns");
     static_assert(NTT % 32 == 0 && NTT >= 32 && NTT <= 256, "MMA N");
-    extern __shared__ __align__(1024) unsigned char smem[];
+    extern __shared__ __align__(128) unsigned char smem[];   // TMA destinations: 128 B; no-swizzle UMMA operands: 16 B
     __shared__ uint64_t bars[2 * NRMAX + 2 * WSTAGES + 1 + Q];
     __shared__ uint32_t tmem_base_s;
     uint64_t* rec_full = bars;
