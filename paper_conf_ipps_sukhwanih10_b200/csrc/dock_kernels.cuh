@@ -665,12 +665,17 @@ __global__ void k_greedy_round(GreedyArgs a)
     if (j > 0 && pk[j - 1] == KEY_MAX) return;   // fewer than j picks possible
     unsigned long long best = KEY_MAX;
     const uint32_t stride = static_cast<uint32_t>(ctas_per_grid) * blockDim.x;
+    float best_s = __int_as_float(0x7f800000);   // score of `best` (float compare first: -0 == +0, no NaN)
     auto consider = [&](uint32_t t, float sv) {
+        if (sv > best_s) return;
         const unsigned long long key = make_key(sv, t);
         if (key >= best) return;
         bool ok = true;
         for (int q = 0; q < j; q++) ok = ok && (cheb_cyc(t, prev[q], a.nx, a.ny, a.nz) > a.rho);
-        if (ok) best = key;
+        if (ok) {
+            best = key;
+            best_s = sv;
+        }
     };
     // four independent loads in flight per thread (the scan is bandwidth-, not compute-bound)
     uint32_t t = part * blockDim.x + threadIdx.x;
