@@ -123,6 +123,21 @@ __device__ __forceinline__ void umma_commit(uint64_t* bar)
 __device__ __forceinline__ void tc_fence_after() { asm volatile("tcgen05.fence::after_thread_sync;" ::: "memory"); }
 __device__ __forceinline__ void tc_fence_before() { asm volatile("tcgen05.fence::before_thread_sync;" ::: "memory"); }
 
+// 32 columns of this warp's TMEM lane quarter; tmem_ld32_nowait leaves the wait::ld to the caller
+__device__ __forceinline__ void tmem_ld32_nowait(uint32_t addr, uint32_t (&v)[32])
+{
+    asm volatile(
+        "tcgen05.ld.sync.aligned.32x32b.x32.b32 {%0,%1,%2,%3,%4,%5,%6,%7,%8,%9,%10,%11,%12,%13,%14,%15,"
+        "%16,%17,%18,%19,%20,%21,%22,%23,%24,%25,%26,%27,%28,%29,%30,%31}, [%32];"
+        : "=r"(v[0]), "=r"(v[1]), "=r"(v[2]), "=r"(v[3]), "=r"(v[4]), "=r"(v[5]), "=r"(v[6]), "=r"(v[7]),
+          "=r"(v[8]), "=r"(v[9]), "=r"(v[10]), "=r"(v[11]), "=r"(v[12]), "=r"(v[13]), "=r"(v[14]), "=r"(v[15]),
+          "=r"(v[16]), "=r"(v[17]), "=r"(v[18]), "=r"(v[19]), "=r"(v[20]), "=r"(v[21]), "=r"(v[22]),
+          "=r"(v[23]), "=r"(v[24]), "=r"(v[25]), "=r"(v[26]), "=r"(v[27]), "=r"(v[28]), "=r"(v[29]),
+          "=r"(v[30]), "=r"(v[31])
+        : "r"(addr));
+}
+__device__ __forceinline__ void tmem_ld_wait() { asm volatile("tcgen05.wait::ld.sync.aligned;" ::: "memory"); }
+
 __device__ __forceinline__ void tmem_ld32(uint32_t addr, uint32_t (&v)[32])
 {
     asm volatile(
@@ -286,6 +301,26 @@ __device__ __forceinline__ void epi_tile(const TcArgs& a, uint32_t tmem, uint64_
         if (a.dbg == 1 || cls >= NCH) {   // diagnostic (no TMEM drain), or no chunk of this row for this class
             __syncwarp();
             if (lane == 0) dk::mbar_arrive(&tm_empty[q]);
+            continue;
+        }
+        if (NCH == 4 && nclass == 2) {
+            // two chunks per warp and row: both loads in flight, one wait, release the row, then score --
+            // the row is free for the next tile's MMAs before any of its values are processed
+            const int c0 = ((q + cls) % NCH) * 32, c1 = ((q + cls + 2) % NCH) * 32;
+            uint32_t v0[32], v1[32];
+            const long long tl0 = tr ? clock64() : 0;
+            const uint32_t base = tmem + (static_cast<uint32_t>(quarter * 32) << 16) + q * NTT;
+            tmem_ld32_nowait(base + c0, v0);
+            tmem_ld32_nowait(base + c1, v1);
+            tmem_ld_wait();
+            if (tr) tw1 += clock64() - tl0;
+            tc_fence_before();
+            __syncwarp();
+            if (lane == 0) dk::mbar_arrive(&tm_empty[q]);
+            if (!row_ok || a.dbg == 2) continue;
+            float* grow = GRID ? a.grid + static_cast<size_t>(slot) * a.nx * a.ny * a.nz + tbase : nullptr;
+            epi_chunk<GRID>(v0, lst, th, th_t, tbase, c0, min(32, a.nx - x0 - c0), grow);
+            epi_chunk<GRID>(v1, lst, th, th_t, tbase, c1, min(32, a.nx - x0 - c1), grow);
             continue;
         }
 #pragma unroll 1
