@@ -390,57 +390,65 @@ dock_status stage_inputs(dock_ctx* ctx, const dock_probe_desc* probes, int n_pro
                          int n_rot, const double** d_xyz, const float** d_coef, const int** d_off,
                          const double** d_rot)
 {
+    // One pinned staging block [off][gather table][rot (host)][host xyz][host coef] goes up in a single
+    // H2D copy; one gather kernel then assembles all probes' atoms (device-resident probe arrays are read
+    // in place).  The host part stays short: until the first launch the GPU idles inside a timed step.
     const int P = ctx->P;
     std::vector<int> off(n_probes + 1, 0);
     for (int i = 0; i < n_probes; i++) off[i + 1] = off[i] + probes[i].n_atoms;
     const int na = off[n_probes];
     const bool rot_dev = is_device_ptr(rot);
-    size_t b_xyz = sizeof(double) * 3 * std::max(na, 1), b_coef = sizeof(float) * P * std::max(na, 1);
-    size_t b_off = sizeof(int) * (n_probes + 1), b_rot = rot_dev ? 0 : sizeof(double) * 9 * n_rot;
+    const size_t b_off = sizeof(int) * (n_probes + 1), b_tab = sizeof(dk::ProbeSrc) * std::max(n_probes, 1);
+    const size_t b_rot = rot_dev ? 0 : sizeof(double) * 9 * n_rot;
+    const size_t b_xyz = sizeof(double) * 3 * std::max(na, 1), b_coef = sizeof(float) * P * std::max(na, 1);
+    const size_t o_tab = (b_off + 15) / 16 * 16, o_rot = o_tab + (b_tab + 15) / 16 * 16;
+    const size_t o_xyz = o_rot + (b_rot + 15) / 16 * 16, o_coef = o_xyz + (b_xyz + 15) / 16 * 16;
+    const size_t total = o_coef + b_coef;
     TRY(ensure(ctx, ctx->xyz, b_xyz));
     TRY(ensure(ctx, ctx->coef, b_coef));
-    TRY(ensure(ctx, ctx->off, b_off));
-    // pinned staging: [off][rot][xyz][coef] (host probes only)
-    size_t o_rot = round_up((int)b_off, 16), o_xyz = o_rot + round_up((int)b_rot, 16);
-    size_t o_coef = o_xyz + b_xyz;
-    TRY(ensure_pinned(ctx, o_coef + b_coef));
+    TRY(ensure(ctx, ctx->off, total));   // device copy of the whole staging block
+    TRY(ensure_pinned(ctx, total));
     // the previous call may still read the staging buffer
     CU(cudaStreamSynchronize(ctx->stream));
     char* hs = static_cast<char*>(ctx->h_stage);
+    char* ds = static_cast<char*>(ctx->off.p);
     memcpy(hs, off.data(), b_off);
-    CU(cudaMemcpyAsync(ctx->off.p, hs, b_off, cudaMemcpyHostToDevice, ctx->stream));
-    if (!rot_dev) {
-        TRY(ensure(ctx, ctx->rot, b_rot));
-        memcpy(hs + o_rot, rot, b_rot);
-        CU(cudaMemcpyAsync(ctx->rot.p, hs + o_rot, b_rot, cudaMemcpyHostToDevice, ctx->stream));
-        *d_rot = static_cast<const double*>(ctx->rot.p);
-    } else {
-        *d_rot = rot;
-    }
+    if (!rot_dev) memcpy(hs + o_rot, rot, b_rot);
+    auto* tab = reinterpret_cast<dk::ProbeSrc*>(hs + o_tab);
     for (int i = 0; i < n_probes; i++) {
         const dock_probe_desc& pr = probes[i];
-        if (pr.n_atoms == 0) continue;
-        double* dx = static_cast<double*>(ctx->xyz.p) + 3 * (size_t)off[i];
-        float* dc = static_cast<float*>(ctx->coef.p) + (size_t)P * off[i];
-        const size_t bx = sizeof(double) * 3 * pr.n_atoms, bc = sizeof(float) * P * pr.n_atoms;
-        if (is_device_ptr(pr.xyz)) {
-            CU(cudaMemcpyAsync(dx, pr.xyz, bx, cudaMemcpyDeviceToDevice, ctx->stream));
-        } else {
-            char* h = hs + o_xyz + sizeof(double) * 3 * (size_t)off[i];
-            memcpy(h, pr.xyz, bx);
-            CU(cudaMemcpyAsync(dx, h, bx, cudaMemcpyHostToDevice, ctx->stream));
+        dk::ProbeSrc t{};
+        t.n = pr.n_atoms;
+        t.off = off[i];
+        if (pr.n_atoms > 0) {
+            const size_t bx = sizeof(double) * 3 * pr.n_atoms, bc = sizeof(float) * P * pr.n_atoms;
+            if (is_device_ptr(pr.xyz)) {
+                t.xyz = pr.xyz;
+            } else {
+                memcpy(hs + o_xyz + sizeof(double) * 3 * (size_t)off[i], pr.xyz, bx);
+                t.xyz = reinterpret_cast<const double*>(ds + o_xyz) + 3 * (size_t)off[i];
+            }
+            if (is_device_ptr(pr.coef)) {
+                t.coef = pr.coef;
+            } else {
+                memcpy(hs + o_coef + sizeof(float) * P * (size_t)off[i], pr.coef, bc);
+                t.coef = reinterpret_cast<const float*>(ds + o_coef) + (size_t)P * off[i];
+            }
         }
-        if (is_device_ptr(pr.coef)) {
-            CU(cudaMemcpyAsync(dc, pr.coef, bc, cudaMemcpyDeviceToDevice, ctx->stream));
-        } else {
-            char* h = hs + o_coef + sizeof(float) * P * (size_t)off[i];
-            memcpy(h, pr.coef, bc);
-            CU(cudaMemcpyAsync(dc, h, bc, cudaMemcpyHostToDevice, ctx->stream));
-        }
+        tab[i] = t;
     }
+    CU(cudaMemcpyAsync(ds, hs, total, cudaMemcpyHostToDevice, ctx->stream));
+    if (n_probes > 0) {
+        dk::k_gather_probes<<<n_probes, 64, 0, ctx->stream>>>(reinterpret_cast<const dk::ProbeSrc*>(ds + o_tab),
+                                                              n_probes, P, static_cast<double*>(ctx->xyz.p),
+                                                              static_cast<float*>(ctx->coef.p));
+        CU(cudaGetLastError());
+        ctx->kernels_last++;
+    }
+    *d_rot = rot_dev ? rot : reinterpret_cast<const double*>(ds + o_rot);
     *d_xyz = static_cast<const double*>(ctx->xyz.p);
     *d_coef = static_cast<const float*>(ctx->coef.p);
-    *d_off = static_cast<const int*>(ctx->off.p);
+    *d_off = reinterpret_cast<const int*>(ds);
     return DOCK_OK;
 }
 

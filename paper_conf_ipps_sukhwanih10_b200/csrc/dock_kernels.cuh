@@ -726,6 +726,31 @@ __global__ void k_fill_u64(unsigned long long* p, size_t n, unsigned long long v
 }
 #endif
 
+// ------------------------------------------------------------------ input staging
+
+// One probe's atoms in the gather table: source pointers (device memory: the caller's buffers or the
+// uploaded staging copy of host arrays), atom count, destination offset.
+struct ProbeSrc {
+    const double* xyz;   // [n][3]
+    const float* coef;   // [n][P]
+    int n, off;
+};
+
+// Gather all probes' atoms into contiguous xyz [na][3] / coef [na][P] (one launch instead of two
+// copies per probe).
+#ifndef DOCK_LAUNCHER_TU   // defined once, in dock.cu
+__global__ void k_gather_probes(const ProbeSrc* __restrict__ tab, int n_probes, int P, double* __restrict__ xyz,
+                                float* __restrict__ coef)
+{
+    const int i = blockIdx.x;
+    if (i >= n_probes) return;
+    const ProbeSrc t = tab[i];
+    for (int j = threadIdx.x; j < 3 * t.n; j += blockDim.x) xyz[3 * static_cast<size_t>(t.off) + j] = t.xyz[j];
+    for (int j = threadIdx.x; j < P * t.n; j += blockDim.x)
+        coef[static_cast<size_t>(P) * t.off + j] = t.coef[j];
+}
+#endif
+
 // ------------------------------------------------------------------ per-call state reset
 
 #ifndef DOCK_LAUNCHER_TU   // defined once, in dock.cu
