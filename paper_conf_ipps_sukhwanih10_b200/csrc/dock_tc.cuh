@@ -42,7 +42,10 @@ constexpr int NEPI_MAX = DOCK_TC_NEPI_MAX;   // epilogue warps: a.nepi in {4, 8}
 constexpr int NTHREADS = (3 + NEPI_MAX) * 32;   // launch bound; both variants launch (3 + a.nepi) * 32 threads
 constexpr int WSTAGES = 16;     // max weight ring depth (runtime a.wstages <= 16; 16 x 4 KB covers the L2 latency)
 constexpr int WCHUNK = 2 * ROT * 16;   // bytes of one K-step of A (2 K-chunks x 128 rotations x 16 B)
-constexpr int KSTEPS = 4;       // K-steps of A per ring stage (one elected issue block of KSTEPS*Q MMAs)
+#ifndef DOCK_TC_KSTEPS
+#define DOCK_TC_KSTEPS 4
+#endif
+constexpr int KSTEPS = DOCK_TC_KSTEPS;   // K-steps of A per ring stage (KSTEPS * Q MMAs per stage)
 constexpr int LIST = 16;        // per-thread candidate list (exact top-LIST keys of one rotation and row class)
 
 struct TcArgs {
