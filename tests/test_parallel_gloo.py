@@ -46,12 +46,13 @@ def _worker(rank, world, port, n_units_cfg, q):
         dist.destroy_process_group()
 
 
-@pytest.mark.parametrize("n_rot", [5, 4])
-def test_sharded_equals_single_rank(orc, n_rot):
+@pytest.mark.parametrize("world,n_rot", [(2, 5), (2, 4), (3, 1)])
+def test_sharded_equals_single_rank(orc, world, n_rot):
+    """(3, 1): 2 units over 3 ranks -- one rank's shard is empty and still joins the all-gather."""
     ctx = mp.get_context("spawn")
     q = ctx.Queue()
     port = _free_port()
-    procs = [ctx.Process(target=_worker, args=(r, 2, port, n_rot, q)) for r in range(2)]
+    procs = [ctx.Process(target=_worker, args=(r, world, port, n_rot, q)) for r in range(world)]
     for p in procs:
         p.start()
     res = dict(q.get(timeout=300) for _ in procs)
@@ -62,7 +63,7 @@ def test_sharded_equals_single_rank(orc, n_rot):
     probes = g.probes(2, 3, 2)
     rot = g.rotations(n_rot)
     ref = _oracle_block(R, g.weights(2), probes, rot, 3, 1, 0, len(probes) * n_rot).numpy()
-    assert np.array_equal(res[0], ref) and np.array_equal(res[1], ref)
+    assert all(np.array_equal(res[r], ref) for r in range(world))
 
 
 def test_shard_ranges_cover_exactly():
