@@ -80,7 +80,8 @@ typedef struct {
     int n_terms;      /* P, number of correlation terms (channels), 1..DOCK_MAX_TERMS */
     int m_max;        /* largest probe grid edge that will be docked, 1..DOCK_MAX_M */
     int device;       /* CUDA device ordinal */
-    float spacing;    /* grid spacing h in Angstrom (> 0); BASELINE uses 0.8 */
+    double spacing;   /* grid spacing h in Angstrom (> 0, finite); BASELINE uses 0.8.  double so that the
+                         kernel divides by exactly the caller's h, as the FP64 oracle does (reading Q18) */
     void* stream;     /* cudaStream_t to run on; NULL => the context creates its own */
 } dock_grid_desc;
 

@@ -10,6 +10,6 @@ Parity status: every function is pinned by tests/test_oracle_pins.py (see DESIGN
 §"Oracle pins").
 """
 from .oracle import (  # noqa: F401
-    build_oracle, check_rotation, voxelize, score_grid, score_at, filter_greedy, dock,
+    build_oracle, check_rotation, voxelize, score_grid, filter_greedy, dock,
     max_threads, OracleError,
 )

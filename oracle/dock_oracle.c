@@ -27,7 +27,8 @@
  *        k = 4 per rotation in FTMap.
  *   4. dock      -- 1-3 for every (probe, rotation) unit, OpenMP over units.
  *
- * Parity pins for every function live in tests/test_oracle_pins.py.
+ * Parity pins for every function live in tests/test_oracle_pins.py (A, the tolerance scale of
+ * every GPU parity check, is pinned by P13).
  */
 #include <math.h>
 #include <stdint.h>
@@ -109,29 +110,6 @@ void orc_score_grid(const float* R, int nx, int ny, int nz, int P, const double*
             }
 }
 
-/* Score (and A) at an explicit list of translations -- same definition as orc_score_grid. */
-void orc_score_at(const float* R, int nx, int ny, int nz, int P, const double* L, int m,
-                  const float* w, const int64_t* t_lin, int n, double* S, double* A)
-{
-    for (int i = 0; i < n; i++) {
-        int64_t t = t_lin[i];
-        int tx = (int)(t % nx), ty = (int)((t / nx) % ny), tz = (int)(t / ((int64_t)nx * ny));
-        double s = 0.0, a = 0.0;
-        for (int p = 0; p < P; p++)
-            for (int vz = 0; vz < m; vz++)
-                for (int vy = 0; vy < m; vy++)
-                    for (int vx = 0; vx < m; vx++) {
-                        double l = L[(((size_t)p * m + vz) * m + vy) * m + vx];
-                        int z = (tz + vz) % nz, y = (ty + vy) % ny, x = (tx + vx) % nx;
-                        double term = (double)w[p] * l * (double)R[(((size_t)p * nz + z) * ny + y) * nx + x];
-                        s += term;
-                        a += fabs(term);
-                    }
-        S[i] = s;
-        if (A) A[i] = a;
-    }
-}
-
 /* Step 3: greedy filter with an N^3 exclusion array.
  * Picks k cells in order; ties in score are broken by the smaller t_lin (reading Q8;
  * -0.0 == +0.0 holds for doubles).  Returns the number of picks made (< k only when
@@ -170,12 +148,15 @@ int orc_filter(const double* S, int nx, int ny, int nz, int k, int rho, int64_t*
  * units ordered probe-major (unit = probe * n_rot + rotation).
  *   probes: xyz_all/coef_all concatenated, atom_off[n_probes+1], m per probe.
  *   out_t  [n_units][k] int64 (-1 when fewer picks), out_s [n_units][k] double,
+ *   out_a  [n_units][k] double or NULL: the magnitude sum A (reading Q16) at each pick,
+ *          the tolerance scale a GPU score is compared with,
  *   out_status [n_units] int (0 or an ORC_E_* code).
  * Uses OpenMP over units when compiled with -fopenmp; n_threads <= 0 => library default. */
 int orc_dock(const float* R, int nx, int ny, int nz, int P, const float* w, double spacing,
              const double* xyz_all, const float* coef_all, const int* atom_off, const int* m_of,
              int n_probes, const double* rot, int n_rot, int64_t unit_begin, int64_t unit_end,
-             int k, int rho, int n_threads, int64_t* out_t, double* out_s, int* out_status)
+             int k, int rho, int n_threads, int64_t* out_t, double* out_s, double* out_a,
+             int* out_status)
 {
     if (unit_begin < 0 || unit_end < unit_begin || unit_end > (int64_t)n_probes * n_rot || k < 1)
         return ORC_E_INVALID;
@@ -191,23 +172,31 @@ int orc_dock(const float* R, int nx, int ny, int nz, int P, const float* w, doub
 #pragma omp parallel
     {
         double* S = (double*)malloc(sizeof(double) * ncell);
+        double* A = out_a ? (double*)malloc(sizeof(double) * ncell) : NULL;
         double* L = (double*)malloc(sizeof(double) * (size_t)P * m_big * m_big * m_big);
 #pragma omp for schedule(dynamic, 1)
         for (int64_t i = 0; i < n_units; i++) {
             int64_t u = unit_begin + i;
             int pr = (int)(u / n_rot), r = (int)(u % n_rot);
             int m = m_of[pr];
-            for (int j = 0; j < k; j++) { out_t[i * k + j] = -1; out_s[i * k + j] = NAN; }
+            for (int j = 0; j < k; j++) {
+                out_t[i * k + j] = -1;
+                out_s[i * k + j] = NAN;
+                if (out_a) out_a[i * k + j] = NAN;
+            }
             int st = orc_check_rotation(rot + 9 * (size_t)r);
             if (st == ORC_OK)
                 st = orc_voxelize(xyz_all + 3 * (size_t)atom_off[pr], coef_all + (size_t)P * atom_off[pr],
                                   atom_off[pr + 1] - atom_off[pr], P, m, rot + 9 * (size_t)r, spacing, L);
             out_status[i] = st;
             if (st != ORC_OK) continue;
-            orc_score_grid(R, nx, ny, nz, P, L, m, w, S, NULL);
-            orc_filter(S, nx, ny, nz, k, rho, out_t + i * k, out_s + i * k);
+            orc_score_grid(R, nx, ny, nz, P, L, m, w, S, A);
+            int np = orc_filter(S, nx, ny, nz, k, rho, out_t + i * k, out_s + i * k);
+            if (out_a)
+                for (int j = 0; j < np; j++) out_a[i * k + j] = A[out_t[i * k + j]];
         }
         free(S);
+        free(A);
         free(L);
     }
     return ORC_OK;

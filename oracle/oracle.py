@@ -42,13 +42,10 @@ def _L():
             lib.orc_voxelize.argtypes = [dp, fp, C.c_int, C.c_int, C.c_int, dp, C.c_double, dp]
             lib.orc_score_grid.argtypes = [fp, C.c_int, C.c_int, C.c_int, C.c_int, dp, C.c_int, fp, dp, dp]
             lib.orc_score_grid.restype = None
-            lib.orc_score_at.argtypes = [fp, C.c_int, C.c_int, C.c_int, C.c_int, dp, C.c_int, fp, lp,
-                                         C.c_int, dp, dp]
-            lib.orc_score_at.restype = None
             lib.orc_filter.argtypes = [dp, C.c_int, C.c_int, C.c_int, C.c_int, C.c_int, lp, dp]
             lib.orc_dock.argtypes = [fp, C.c_int, C.c_int, C.c_int, C.c_int, fp, C.c_double,
                                      dp, fp, ip, ip, C.c_int, dp, C.c_int, C.c_int64, C.c_int64,
-                                     C.c_int, C.c_int, C.c_int, lp, dp, ip]
+                                     C.c_int, C.c_int, C.c_int, lp, dp, dp, ip]
             lib.orc_max_threads.argtypes = []
             _lib = lib
     return _lib
@@ -100,16 +97,6 @@ def score_grid(R: np.ndarray, L: np.ndarray, w: np.ndarray, with_A: bool = True)
     return (S, A) if with_A else S
 
 
-def score_at(R: np.ndarray, L: np.ndarray, w: np.ndarray, t_lin: Sequence[int]) -> Tuple[np.ndarray, np.ndarray]:
-    R, L, w = _f32(R), _f64(L), _f32(w)
-    P, nz, ny, nx = R.shape
-    t = np.ascontiguousarray(t_lin, dtype=np.int64).reshape(-1)
-    S = np.empty(t.shape[0]); A = np.empty(t.shape[0])
-    _L().orc_score_at(_p(R, C.c_float), nx, ny, nz, P, _p(L, C.c_double), L.shape[-1], _p(w, C.c_float),
-                      _p(t, C.c_int64), t.shape[0], _p(S, C.c_double), _p(A, C.c_double))
-    return S, A
-
-
 def filter_greedy(S: np.ndarray, k: int, rho: int) -> Tuple[np.ndarray, np.ndarray]:
     """Greedy best-then-exclude filter: (t_lin[k'], score[k'])."""
     S = _f64(S)
@@ -122,8 +109,9 @@ def filter_greedy(S: np.ndarray, k: int, rho: int) -> Tuple[np.ndarray, np.ndarr
 
 
 def dock(R: np.ndarray, w: np.ndarray, spacing: float, probes, rot: np.ndarray, k: int, rho: int,
-         unit_begin: int = 0, unit_end: int | None = None, n_threads: int = 0):
-    """Full docking over probe-major (probe, rotation) units -> (t_lin [U][k], score [U][k], status [U])."""
+         unit_begin: int = 0, unit_end: int | None = None, n_threads: int = 0, with_A: bool = False):
+    """Full docking over probe-major (probe, rotation) units -> (t_lin [U][k], score [U][k], status [U]),
+    and with ``with_A`` also the magnitude sum A [U][k] at each pick (reading Q16)."""
     R, w, rot = _f32(R), _f32(w), _f64(rot).reshape(-1, 9)
     P, nz, ny, nx = R.shape
     n_rot = rot.shape[0]
@@ -137,11 +125,13 @@ def dock(R: np.ndarray, w: np.ndarray, spacing: float, probes, rot: np.ndarray, 
     U = unit_end - unit_begin
     out_t = np.full((U, k), -1, dtype=np.int64)
     out_s = np.full((U, k), np.nan)
+    out_a = np.full((U, k), np.nan) if with_A else None
     st = np.zeros(U, dtype=np.int32)
     rc = _L().orc_dock(_p(R, C.c_float), nx, ny, nz, P, _p(w, C.c_float), float(spacing),
                        _p(xyz, C.c_double), _p(coef, C.c_float), _p(off, C.c_int), _p(ms, C.c_int),
                        len(probes), _p(rot, C.c_double), n_rot, unit_begin, unit_end, k, rho, n_threads,
-                       _p(out_t, C.c_int64), _p(out_s, C.c_double), _p(st, C.c_int))
+                       _p(out_t, C.c_int64), _p(out_s, C.c_double),
+                       _p(out_a, C.c_double) if with_A else None, _p(st, C.c_int))
     if rc != 0:
         raise OracleError(f"dock status {rc}")
-    return out_t, out_s, st
+    return (out_t, out_s, st, out_a) if with_A else (out_t, out_s, st)

@@ -36,7 +36,7 @@ class dock_pose(C.Structure):
 
 class dock_grid_desc(C.Structure):
     _fields_ = [("nx", C.c_int), ("ny", C.c_int), ("nz", C.c_int), ("n_terms", C.c_int), ("m_max", C.c_int),
-                ("device", C.c_int), ("spacing", C.c_float), ("stream", C.c_void_p)]
+                ("device", C.c_int), ("spacing", C.c_double), ("stream", C.c_void_p)]
 
 
 class dock_probe_desc(C.Structure):

@@ -58,7 +58,7 @@ struct dock_ctx {
     cudaStream_t stream = nullptr;
     bool own_stream = false;
     int nx = 0, ny = 0, nz = 0, P = 0, m_max = 0;
-    float spacing = 0.f;
+    double spacing = 0.0;   // h exactly as given (the kernel divides by it in FP64, like the oracle)
     int n_sms = 148;
     double l2_bytes = 0;
     dk::Geo geo{};
@@ -544,9 +544,14 @@ dock_status run_grid(dock_ctx* ctx, int m, int n_slots, const float* Lw, float* 
     return DOCK_OK;
 }
 
-// Exact fallback for flagged slots: full score grid + exact greedy.
+dock_status run_grid_tc(dock_ctx* ctx, int m, int n_slots, const float* Lw, float* grid);
+
+// Exact fallback for flagged slots: full score grid + exact greedy.  The grids come from the
+// engine that produced the candidates (use_tc: the tcgen05 GRID epilogue; else the FFMA one), so a
+// rotation's score bits never depend on whether it was flagged.
 dock_status run_fallback(dock_ctx* ctx, int m, int nfb, int64_t unit_begin, int n_rot, const double* xyz,
-                         const float* coef, const int* off, const double* rot, int k, int rho, void* poses)
+                         const float* coef, const int* off, const double* rot, int k, int rho, void* poses,
+                         bool use_tc)
 {
     std::vector<int> slots(nfb);
     CU(cudaMemcpyAsync(slots.data(), ctx->fb_list.p, sizeof(int) * nfb, cudaMemcpyDeviceToHost, ctx->stream));
@@ -573,7 +578,10 @@ dock_status run_fallback(dock_ctx* ctx, int m, int nfb, int64_t unit_begin, int 
         const int* d_outslot = d_units + chunk;
         TRY(run_voxelize(ctx, m, n, 0, d_units, n_rot, xyz, coef, off, rot, ctx->d_w,
                          static_cast<float*>(ctx->Lw_fb.p)));
-        TRY(run_grid(ctx, m, n, static_cast<const float*>(ctx->Lw_fb.p), static_cast<float*>(ctx->grid.p)));
+        if (use_tc)
+            TRY(run_grid_tc(ctx, m, n, static_cast<const float*>(ctx->Lw_fb.p), static_cast<float*>(ctx->grid.p)));
+        else
+            TRY(run_grid(ctx, m, n, static_cast<const float*>(ctx->Lw_fb.p), static_cast<float*>(ctx->grid.p)));
         dk::GreedyArgs ga{};
         ga.grid = static_cast<const float*>(ctx->grid.p);
         ga.slots = d_outslot;
@@ -808,7 +816,7 @@ dock_status dock_init(const dock_grid_desc* g, const float* receptor, const floa
     if (!out) return DOCK_E_INVALID_ARG;
     *out = nullptr;
     if (!g || !receptor || !weights) return DOCK_E_INVALID_ARG;
-    if (g->nx < 1 || g->ny < 1 || g->nz < 1 || g->n_terms < 1 || g->m_max < 1 || !(g->spacing > 0.f) ||
+    if (g->nx < 1 || g->ny < 1 || g->nz < 1 || g->n_terms < 1 || g->m_max < 1 || !(g->spacing > 0.0) ||
         !std::isfinite(g->spacing))
         return DOCK_E_INVALID_ARG;
     if (g->n_terms > DOCK_MAX_TERMS || g->m_max > DOCK_MAX_M) return DOCK_E_UNSUPPORTED;
@@ -1210,7 +1218,7 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
     ctx->fallback_last = nfb;
     ctx->cand_max_last = (unsigned)ctx->h_small[2];
     if (nfb > 0)
-        TRY(run_fallback(ctx, m, nfb, unit_begin, n_rot, d_xyz, d_coef, d_off, d_rot, k, rho, d_poses));
+        TRY(run_fallback(ctx, m, nfb, unit_begin, n_rot, d_xyz, d_coef, d_off, d_rot, k, rho, d_poses, use_tc));
     if (!out_dev)
         CU(cudaMemcpyAsync(out, d_poses, sizeof(dock_pose) * (size_t)n_units * k, cudaMemcpyDeviceToHost,
                            ctx->stream));

@@ -52,6 +52,40 @@ def test_struct_layouts():
     assert ctypes.sizeof(N.dock_grid_desc) == 40
 
 
+def test_struct_layouts_match_header(tmp_path):
+    """Every ctypes struct of the binding has the sizes and field offsets that include/dock.h gives a
+    C compiler (catches a field whose type changed on one side only, e.g. the spacing's width)."""
+    import shutil
+    import subprocess
+    from paper_conf_ipps_sukhwanih10_b200 import _native as N
+    cc = shutil.which("gcc") or shutil.which("cc")
+    if not cc:
+        pytest.skip("no C compiler")
+    structs = {"dock_pose": N.dock_pose, "dock_grid_desc": N.dock_grid_desc,
+               "dock_probe_desc": N.dock_probe_desc, "dock_info": N.dock_info}
+    lines = ['#include <stdio.h>', '#include <stddef.h>', '#include "dock.h"', "int main(void) {"]
+    for name, cls in structs.items():
+        lines.append(f'printf("{name} size %zu\\n", sizeof({name}));')
+        for f, _ in cls._fields_:
+            lines.append(f'printf("{name} {f} %zu\\n", offsetof({name}, {f}));')
+            lines.append(f'printf("{name} {f}.size %zu\\n", sizeof((({name}*)0)->{f}));')
+    lines.append("return 0; }")
+    src = tmp_path / "layout.c"
+    src.write_text("\n".join(lines))
+    exe = tmp_path / "layout"
+    root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+    subprocess.check_call([cc, "-std=c99", "-I", os.path.join(root, "include"), "-o", str(exe), str(src)])
+    got = {}
+    for line in subprocess.check_output([str(exe)], text=True).splitlines():
+        a, b, c = line.split()
+        got[(a, b)] = int(c)
+    for name, cls in structs.items():
+        assert got[(name, "size")] == ctypes.sizeof(cls), name
+        for f, _ in cls._fields_:
+            assert got[(name, f)] == getattr(cls, f).offset, f"{name}.{f}"
+            assert got[(name, f + ".size")] == getattr(cls, f).size, f"{name}.{f} width"
+
+
 def test_sass_is_sm100a_with_tma():
     """The hot kernel is compiled for sm_100a and issues TMA (UTMALDG) + bulk copies (UBLKCP)."""
     import shutil

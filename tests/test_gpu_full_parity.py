@@ -1,0 +1,102 @@
+"""Full-workload GPU parity: EVERY unit of BASELINE configs[1] (c64, 500 units) and configs[2] (prod,
+16 probes x 500 rotations = 8000 units) against the FP64 oracle.
+
+The oracle's picks, scores S and magnitude sums A (reading Q16) for every unit are precomputed by
+scripts/oracle_cache.py (which calls only oracle/) and stored in tests/golden/oracle_<cfg>_k4_rho1.npz,
+keyed by a hash of the generated inputs.  The GPU docks the whole workload in the launch configuration
+bench.py times (device-resident inputs and poses, one dock_probe_batch).  A unit whose picks equal the
+oracle's must report scores within 1e-4 * A; a unit whose picks differ is re-scored in full by the oracle
+and checked by the tie-aware validator (tests/validator.py, reading Q17).  The achieved max |err|/A and the
+number of tie-divergent units are printed and appended to gpurun_out/parity_margins.jsonl.
+"""
+import concurrent.futures as cf
+import json
+import os
+import sys
+
+import numpy as np
+import pytest
+
+import dockgen as g
+from validator import validate_unit
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+sys.path.insert(0, os.path.join(ROOT, "scripts"))
+import oracle_cache  # noqa: E402  (input generation + hash only; no arithmetic of the method)
+
+pytestmark = pytest.mark.gpu
+H = g.SPACING
+ENGINES = [1, 2, 3]   # 1 FP32 FFMA, 2 tcgen05 variant 1, 3 tcgen05 variant 2
+
+
+@pytest.fixture(scope="module")
+def D():
+    import torch
+    assert torch.cuda.is_available(), "GPU tests need a CUDA device"
+    from paper_conf_ipps_sukhwanih10_b200 import build
+    build.build_native()
+    import paper_conf_ipps_sukhwanih10_b200 as D
+    return D
+
+
+def _record(entry):
+    print("PARITY_MARGIN " + json.dumps(entry))
+    out = os.path.join(ROOT, "gpurun_out")
+    if os.path.isdir(out):
+        with open(os.path.join(out, "parity_margins.jsonl"), "a") as f:
+            f.write(json.dumps(entry) + "\n")
+
+
+@pytest.mark.parametrize("engine", ENGINES)
+@pytest.mark.parametrize("cfg", ["c64", "prod"])
+def test_full_workload_parity(D, orc, cfg, engine):
+    import torch
+    k, rho = 4, 1
+    path = oracle_cache.cache_path(cfg, k, rho)
+    assert os.path.exists(path), f"missing {path}: run scripts/oracle_cache.py --config {cfg}"
+    ref = np.load(path)
+    c, R, w, probes, rot = oracle_cache.inputs(cfg)
+    assert str(ref["input_hash"]) == oracle_cache.input_hash(R, w, probes, rot, k, rho), "inputs changed"
+    assert (ref["status"] == 0).all()
+    dev = torch.device("cuda", 0)
+    ctx = D.dock_init(torch.from_numpy(R).to(dev), torch.from_numpy(w).to(dev), H, m_max=c.m, device=0)
+    D.dock_set_tuning(ctx, D.DOCK_TUNE_ENGINE, 1 if engine == 1 else 2)
+    if engine >= 2:
+        D.dock_set_tuning(ctx, D.DOCK_TUNE_TC_VARIANT, engine - 1)
+    n = c.n_probes * c.n_rot
+    dprobes = [{"xyz": torch.from_numpy(p.xyz).to(dev), "coef": torch.from_numpy(p.coef).to(dev), "m": p.m}
+               for p in probes]
+    out = torch.empty((n, k, 4), dtype=torch.int32, device=dev)
+    D.dock_probe_batch(ctx, dprobes, torch.from_numpy(rot).to(dev), 0, n, k, rho, out=out)
+    torch.cuda.synchronize()
+    info = D.dock_get_info(ctx)
+    ctx.close()
+    eng = 1 if info["engine_last"] == 1 else 1 + info["tc_variant_last"]
+    assert eng == engine
+    poses = D.poses_from_device(out)
+    assert (poses["rot"] == np.arange(n)[:, None] % c.n_rot).all()
+    t_g = poses["t_lin"].astype(np.int64)
+    s_g = poses["score"].astype(np.float64)
+    same = (t_g == ref["t_lin"]).all(axis=1)
+    err = np.abs(s_g - ref["score"])
+    rel = err / np.maximum(ref["A"], 1e-30)
+    bad = same[:, None] & (err > 1e-4 * ref["A"] + 1e-12)
+    assert not bad.any(), f"{int(bad.sum())} picks outside 1e-4*A; max err/A {rel[same].max()}"
+    div = np.flatnonzero(~same)
+
+    def check(u):
+        pr, r = probes[u // c.n_rot], u % c.n_rot
+        L = orc.voxelize(pr.xyz, pr.coef, pr.m, rot[r], H)
+        S, A = orc.score_grid(R, L, w)
+        validate_unit(S, A, t_g[u], poses[u]["score"], k, rho)
+        tt = t_g[u]
+        return float(np.max(np.abs(s_g[u] - S.reshape(-1)[tt]) / np.maximum(A.reshape(-1)[tt], 1e-30)))
+
+    threads = max(1, min(32, len(os.sched_getaffinity(0))))
+    with cf.ThreadPoolExecutor(threads) as ex:
+        div_rel = list(ex.map(check, div.tolist()))
+    max_rel = max([float(rel[same].max()) if same.any() else 0.0] + div_rel)
+    _record({"config": cfg, "engine": engine, "units": n, "units_identical_picks": int(same.sum()),
+             "units_tie_divergent_validated": int(len(div)), "max_err_over_A": max_rel,
+             "fallback_rotations": int(info["fallback_last"]), "tolerance": 1e-4})
+    assert max_rel <= 1e-4

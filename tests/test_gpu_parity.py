@@ -77,6 +77,81 @@ def test_voxelize_matches_oracle(D, orc, m):
     ctx.close()
 
 
+def _golden_voxel_cases():
+    import os
+    path = os.path.join(os.path.dirname(__file__), "golden", "voxelize_cases.txt")
+    for line in open(path):
+        if line.startswith("#") or not line.strip():
+            continue
+        m, x, v = line.split()
+        yield int(m), float(x), int(v)
+
+
+def test_voxelize_golden_cases_on_gpu(D):
+    """tests/golden/voxelize_cases.txt (reading Q3) replayed through the C ABI on
+    all three axes: dock_voxelize must put the atom on the hand-derived voxel, and both dock_voxelize
+    and the hot path (dock_probe) must return DOCK_E_PROBE_OUTSIDE_GRID for the rows marked -1."""
+    ctx = D.dock_init(g.receptor_uniform((16, 16, 16), 1), np.ones(1, np.float32), H, m_max=4)
+    for m, x, v in _golden_voxel_cases():
+        for axis in range(3):
+            xyz = np.zeros((1, 3))
+            xyz[0, axis] = x
+            pr = g.Probe(xyz, np.ones((1, 1), np.float32), m)
+            eye = np.eye(3).reshape(1, 9)
+            if v < 0:
+                with pytest.raises(D.DockError) as e:
+                    D.dock_voxelize(ctx, pr, eye)
+                assert e.value.status == -3, (m, x, axis)
+                with pytest.raises(D.DockError) as e:
+                    D.dock_probe(ctx, pr, eye, k=1, rho=0)
+                assert e.value.status == -3, (m, x, axis)
+                continue
+            L = D.dock_voxelize(ctx, pr, eye)
+            c = int(np.floor((m - 1) / 2.0 + 0.5))
+            want = [c, c, c]
+            want[axis] = v
+            assert np.argwhere(L[0, 0] != 0).tolist() == [[want[2], want[1], want[0]]], (m, x, axis)
+    ctx.close()
+
+
+@pytest.mark.parametrize("m", [2, 3, 4, 5, 8])
+def test_voxelize_half_voxel_boundaries_bitwise(D, orc, m):
+    """Atoms placed so that Q x / h lands within 1e-9 A of a rounding boundary (k + 1/2 - c) under random
+    rotations: the GPU's voxel indices equal the FP64 oracle's bit for bit (reading Q18).  An FP32 copy of
+    h (0.8f = 0.800000011920929) would move g by ~2e-8 and flip these cases."""
+    rng = np.random.default_rng(1800 + m)
+    P = 1
+    ctx = D.dock_init(g.receptor_uniform((16, 16, 16), P), np.ones(P, np.float32), H, m_max=8)
+    rot = g.rotations(24, seed=77)
+    c = (m - 1) / 2.0
+    n_checked = 0
+    for r in range(len(rot)):
+        Q = rot[r].reshape(3, 3)
+        atoms = []
+        for a in range(8):
+            y = (rng.integers(0, m, 3) - c) * H              # voxel centres ...
+            axis = int(rng.integers(0, 3))
+            kk = int(rng.integers(0, m - 1))
+            eps = float(rng.choice([-1e-9, 0.0, 1e-9]))
+            y[axis] = (kk + 0.5 - c) * H + eps               # ... with one coordinate on a boundary
+            atoms.append(Q.T @ y)                            # so that Q x = y up to rounding
+        xyz = np.array(atoms)
+        coef = (2.0 ** np.arange(len(atoms))).astype(np.float32).reshape(-1, 1)   # exact sums identify atoms
+        pr = g.Probe(xyz, coef, m)
+        try:
+            Lo = orc.voxelize(xyz, coef, m, rot[r], H)
+        except orc.OracleError:
+            with pytest.raises(D.DockError) as e:
+                D.dock_voxelize(ctx, pr, rot[r:r + 1])
+            assert e.value.status == -3
+            continue
+        Lg = D.dock_voxelize(ctx, pr, rot[r:r + 1])[0]
+        assert np.array_equal(Lg.astype(np.float64), Lo), f"rotation {r}"
+        n_checked += 1
+    assert n_checked >= len(rot) // 2
+    ctx.close()
+
+
 # ----------------------------------------------------------------------------- score grids
 
 
@@ -214,17 +289,20 @@ def test_integer_inputs_exact_poses(D, orc, rho, k, engine):
     assert np.array_equal(poses["score"].astype(np.float64), s_o)
 
 
-def test_fallback_path_identical(D):
-    """The exact full-grid fallback returns the same poses (bitwise) as the candidate path
-    (both use the FFMA arithmetic here)."""
+@pytest.mark.parametrize("engine", ENGINES)
+def test_fallback_path_identical(D, engine):
+    """The exact full-grid fallback returns the same poses (bitwise: t_lin and score bits) as the
+    candidate path, on every engine: the fallback's score grids come from the engine that produced the
+    candidates (tcgen05 GRID epilogue for engines 2/3, FFMA for engine 1)."""
     P, m = 4, 4
     R = g.receptor_ftmap_like((48, 40, 36), P)
     w = g.weights(P)
     probes = g.probes(2, m, P)
     rot = g.rotations(13)
-    ctx = _ctx(D, R, w, m, 1)
+    ctx = _ctx(D, R, w, m, engine)
     for rho in (0, 1):
         a = D.dock_probe_batch(ctx, probes, rot, k=4, rho=rho)
+        assert _engine_id(D.dock_get_info(ctx)) == engine
         D.dock_set_tuning(ctx, D.DOCK_TUNE_FORCE_FALLBACK, 1)
         b = D.dock_probe_batch(ctx, probes, rot, k=4, rho=rho)
         assert D.dock_get_info(ctx)["fallback_last"] == len(probes) * len(rot)
@@ -254,8 +332,10 @@ def test_invariance_batch_shard_launch(D, engine):
         D.dock_set_tuning(ctx, D.DOCK_TUNE_REGIONS, G)
         assert np.array_equal(D.dock_probe_batch(ctx, probes, rot, k=4, rho=1), ref)
     D.dock_set_tuning(ctx, D.DOCK_TUNE_REGIONS, 0)
-    D.dock_set_tuning(ctx, D.DOCK_TUNE_CAND_CAP, 32)
-    assert np.array_equal(D.dock_probe_batch(ctx, probes, rot, k=4, rho=1)["t_lin"], ref["t_lin"])
+    D.dock_set_tuning(ctx, D.DOCK_TUNE_CAND_CAP, 32)   # small cap: overflowing rotations take the fallback
+    capped = D.dock_probe_batch(ctx, probes, rot, k=4, rho=1)
+    assert np.array_equal(capped["t_lin"], ref["t_lin"])
+    assert np.array_equal(capped["score"].view(np.uint32), ref["score"].view(np.uint32))
     D.dock_set_tuning(ctx, D.DOCK_TUNE_CAND_CAP, 1024)
     # reversed rotation order: per-rotation results follow the rotation
     rev = rot[::-1].copy()

@@ -110,6 +110,59 @@ def test_P3_conv3d_library(orc):
         assert np.max(np.abs(S - ref)) <= 1e-9 * max(1.0, A.max())
 
 
+# ----------------------------------------------------------------------------- P13 (the tolerance scale A)
+
+
+def test_P13_magnitude_sum_conv3d_library(orc):
+    """A[t] = sum_p sum_v |w_p L_p[v] R_p[(t+v) mod n]| (reading Q16) -- the scale of every GPU
+    tolerance -- equals a library convolution of |R| (circular padding) with |w_p L_p|."""
+    torch = pytest.importorskip("torch")
+    import torch.nn.functional as F
+    rng = np.random.default_rng(131)
+    for shape, m, P in [((12, 10, 9), 4, 4), ((9, 11, 7), 3, 2), ((8, 8, 8), 5, 3)]:
+        R = g.receptor_uniform(shape, P, seed=13)
+        L = _rand_L(rng, P, m, 0.5)
+        w = np.array([1.0, -0.6, 2.5, 0.4][:P], np.float32)   # signs and |w| != 1: a dropped |w_p| fails
+        S, A = orc.score_grid(R, L, w)
+        x = torch.from_numpy(np.abs(R.astype(np.float64)))[None]
+        x = F.pad(x, (0, m - 1, 0, m - 1, 0, m - 1), mode="circular")
+        k = torch.from_numpy(np.abs(L * w.astype(np.float64)[:, None, None, None]))[None]
+        ref = F.conv3d(x, k)[0, 0].numpy()
+        assert np.max(np.abs(A - ref)) <= 1e-12 * A.max()
+        assert (A >= np.abs(S) - 1e-12 * A.max()).all()          # triangle inequality
+
+
+def test_P13_magnitude_sum_single_atom_exact(orc):
+    """One atom with coefficients c on voxel v0: A = sum_p |w_p c_p| roll(|R_p|, -v0), bitwise for P = 1;
+    and for same-sign terms A == |S| (no cancellation)."""
+    R = g.receptor_uniform((9, 8, 7), 2, seed=14)
+    for m, v0 in [(3, (2, 0, 1)), (4, (1, 3, 2))]:
+        pr = g.voxel_centre_probe([v0], m, 1, coef=np.array([[-1.75]], np.float32))
+        L = orc.voxelize(pr.xyz, pr.coef, m, np.eye(3).reshape(9), H)
+        w = np.array([0.6], np.float32)
+        _, A = orc.score_grid(R[:1], L, w)
+        want = (abs(np.float64(w[0])) * 1.75) * np.abs(R[0].astype(np.float64))
+        assert np.array_equal(A, np.roll(want, (-v0[2], -v0[1], -v0[0]), axis=(0, 1, 2)))
+    Rp = np.abs(R)
+    L = np.abs(_rand_L(np.random.default_rng(5), 2, 3, 0.6))
+    S, A = orc.score_grid(Rp, L, np.array([0.5, 2.0], np.float32))
+    assert np.max(np.abs(A - S)) <= 1e-12 * A.max()
+
+
+def test_P13_dock_reports_A_at_picks(orc):
+    """orc_dock's per-pick A is the score grid's A at the picked cells."""
+    R = g.receptor_uniform((10, 9, 8), 3, seed=15)
+    w = g.weights(3)
+    pr = g.probe(1, 3, 3)
+    rot = g.rotations(3)
+    t, s, st, a = orc.dock(R, w, H, [pr], rot, 4, 1, with_A=True)
+    assert (st == 0).all()
+    for r in range(3):
+        S, A = orc.score_grid(R, orc.voxelize(pr.xyz, pr.coef, 3, rot[r], H), w)
+        assert np.array_equal(a[r], A.reshape(-1)[t[r]])
+        assert np.array_equal(s[r], S.reshape(-1)[t[r]])
+
+
 # ----------------------------------------------------------------------------- P4/P5
 
 
