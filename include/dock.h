@@ -21,7 +21,11 @@
  *             Chebyshev ball of radius rho around each pick (Q9: rho = 1 is the
  *             paper-faithful default, rho = 0 is plain top-k).
  *   - t_lin = (tz*ny + ty)*nx + tx; x is the fastest axis everywhere.
- * GPU arithmetic is FP32 FMA (Q15); the FP64 oracle (oracle/) is the reference.
+ * GPU arithmetic (reading Q15): engine 1 is FP32 FFMA; the default tcgen05 engine multiplies bf16
+ * hi/lo splits of both operands (x = hi + lo, bf16x3: Rhi*Whi + Rlo*Whi + Rhi*Wlo) and accumulates
+ * in FP32 -- the dropped Rlo*Wlo and the lo roundings bound the error by ~3*2^-18 relative per term,
+ * i.e. ~1e-5*A against the 1e-4*A tolerance (reading Q16); integer-valued inputs stay exact.  The
+ * FP64 oracle (oracle/) is the reference.
  *
  * Conventions
  *   - Every call returns dock_status (DOCK_OK = 0); no exception crosses the ABI.
@@ -29,9 +33,15 @@
  *     cudaPointerGetAttributes.  The library never takes ownership of caller memory:
  *     dock_init copies the receptor and weights; probe/rotation inputs are only read
  *     during the call.
- *   - All work runs on the context's stream.  Calls that produce results return after
- *     that stream has been synchronized (results are then valid in host or device
- *     output memory).
+ *   - All work runs on the context's stream.  dock_probe / dock_probe_batch with a DEVICE
+ *     output pointer are asynchronous: they enqueue the whole hot path (including the exact
+ *     fallback, whose loop is driven by a device-side flag count) and return without any host
+ *     synchronisation; the poses are valid once the context's stream reaches that point (e.g.
+ *     after dock_sync, or for any later work ordered on the stream such as an NCCL all-gather).
+ *     Device-detected input errors (DOCK_E_BAD_ROTATION, DOCK_E_PROBE_OUTSIDE_GRID) of an
+ *     asynchronous call are sticky and reported by the next sync point: dock_sync, or the next
+ *     call with host output / dock_score_grid / dock_voxelize.  Calls with HOST output (and the
+ *     debug calls) synchronise the stream before returning.
  *   - A context is bound to one device and one stream and is not thread-safe.
  *     After DOCK_E_CUDA the context is unusable and must be destroyed.
  */
@@ -118,6 +128,12 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
                              const double* rot, int n_rot, int64_t unit_begin, int64_t unit_end,
                              int k, int rho, dock_pose* out);
 
+/* dock_sync -- sync point of the asynchronous calls: waits for the context's stream, returns the
+ * first device-detected error of the calls since the previous sync point (DOCK_E_BAD_ROTATION,
+ * DOCK_E_PROBE_OUTSIDE_GRID; cleared by this call) or DOCK_E_CUDA, and makes the last call's
+ * statistics (fallback_last, cand_max_last) available to dock_get_info. */
+dock_status dock_sync(dock_ctx* ctx);
+
 /* dock_score_grid -- test/debug: the full weighted score grid of one rotated probe.
  *   rot9     : [9] float64 rotation, host or device.
  *   out      : [nz][ny][nx] float32 S (weighted), host or device.
@@ -155,8 +171,8 @@ typedef struct {
     int lanes_x, tile_x, tile_y, tile_z, n_tiles, n_stages, smem_bytes;
     int regions_last;          /* regions used by the last dock_probe_batch */
     int64_t items_last;        /* CTAs (rotation batch x region) launched by the last call */
-    int64_t fallback_last;     /* rotations that took the exact fallback in the last call */
-    int64_t cand_max_last;     /* largest candidate count of one rotation in the last call */
+    int64_t fallback_last;     /* rotations that took the exact fallback in the last call (valid after its sync point) */
+    int64_t cand_max_last;     /* largest candidate count of one rotation in the last call (idem) */
     int64_t kernels_last;      /* kernels launched by the last call */
     int rot_batch;             /* rotations per register block (RB) */
     int x_per_thread;          /* translations along x per thread (XT) */
@@ -170,6 +186,8 @@ typedef struct {
     int tc_ksteps_last;        /* K-steps (K = 16 each) per translation row executed by the last tcgen05 launch */
     int tc_row_last;           /* translations per MMA row (MMA N) of the last tcgen05 launch */
     int tc_rows_per_tile_last; /* translation rows per tile (TMEM accumulators) of the last tcgen05 launch */
+    int pending;               /* 1 if the last asynchronous call has not reached a sync point (dock_sync) */
+    int fb_chunk;              /* flagged rotations per iteration of the device-driven fallback loop */
 } dock_info;
 
 dock_status dock_get_info(const dock_ctx* ctx, dock_info* info);

@@ -52,10 +52,11 @@ class dock_info(C.Structure):
                 ("padded_z", C.c_int), ("l2_bytes", C.c_double), ("corr_ms_last", C.c_double),
                 ("n_sms", C.c_int), ("engine_last", C.c_int), ("tc_available", C.c_int),
                 ("tc_variant_last", C.c_int), ("tc_ksteps_last", C.c_int),
-                ("tc_row_last", C.c_int), ("tc_rows_per_tile_last", C.c_int)]
+                ("tc_row_last", C.c_int), ("tc_rows_per_tile_last", C.c_int), ("pending", C.c_int),
+                ("fb_chunk", C.c_int)]
 
 
-EXPORTS = ["dock_init", "dock_probe", "dock_probe_batch", "dock_score_grid", "dock_voxelize",
+EXPORTS = ["dock_init", "dock_probe", "dock_probe_batch", "dock_sync", "dock_score_grid", "dock_voxelize",
            "dock_set_tuning", "dock_get_info", "dock_destroy", "dock_status_string", "dock_last_error"]
 
 _lib = None
@@ -73,6 +74,7 @@ def lib() -> C.CDLL:
     L.dock_init.argtypes = [C.POINTER(dock_grid_desc), vp, vp, C.POINTER(vp)]
     L.dock_probe.argtypes = [vp, C.POINTER(dock_probe_desc), vp, i, i, i, vp]
     L.dock_probe_batch.argtypes = [vp, C.POINTER(dock_probe_desc), i, vp, i, i64, i64, i, i, vp]
+    L.dock_sync.argtypes = [vp]
     L.dock_score_grid.argtypes = [vp, C.POINTER(dock_probe_desc), vp, vp, vp]
     L.dock_voxelize.argtypes = [vp, C.POINTER(dock_probe_desc), vp, i, vp]
     L.dock_set_tuning.argtypes = [vp, i, i64]
@@ -83,7 +85,7 @@ def lib() -> C.CDLL:
     L.dock_status_string.restype = C.c_char_p
     L.dock_last_error.argtypes = [vp]
     L.dock_last_error.restype = C.c_char_p
-    for name in ("dock_init", "dock_probe", "dock_probe_batch", "dock_score_grid", "dock_voxelize",
+    for name in ("dock_init", "dock_probe", "dock_probe_batch", "dock_sync", "dock_score_grid", "dock_voxelize",
                  "dock_set_tuning", "dock_get_info"):
         getattr(L, name).restype = C.c_int
     _lib = L

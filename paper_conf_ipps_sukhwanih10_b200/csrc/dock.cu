@@ -88,10 +88,27 @@ struct dock_ctx {
     int tc_dbg = 0;
     // per-call scratch (grow-only)
     DevBuf xyz, coef, off, rot, Lw, T, mu, cnt, cand, poses, fb_list, grid, slots, units, Lw_fb, picks;
-    int* d_small = nullptr;    // [0] status, [1] fb_cnt, [2] cand_max
-    int* h_small = nullptr;    // pinned mirror
-    void* h_stage = nullptr;   // pinned staging for host inputs
+    int* d_small = nullptr;    // [0] status bits (sticky until the next sync point), [1] fb_cnt, [2] cand_max
+    int* h_small = nullptr;    // pinned mirror, written by the async copy at the end of every call
+    void* h_stage = nullptr;   // pinned scratch of the synchronous FFT comparison engine
     size_t h_stage_cap = 0;
+    // pinned staging ring for the per-call inputs: a slot is rewritten only after the H2D copy that last
+    // read it has executed (its event), so calls never wait for the GPU to drain
+    struct Stage {
+        void* h = nullptr;
+        size_t cap = 0;
+        cudaEvent_t ev = nullptr;
+        bool live = false;
+    } stage[3];
+    int stage_next = 0;
+    // asynchronous calls: end-of-call event (status copied to h_small), unsynced flag
+    cudaEvent_t ev_done = nullptr;
+    bool unsynced = false;
+    // device-driven exact fallback (a CUDA graph with a WHILE node over chunks of flagged slots)
+    cudaStream_t cap_stream = nullptr, cap_stream2 = nullptr;   // private capture streams
+    cudaGraphExec_t fb_exec = nullptr;
+    unsigned char fb_key[128] = {0};
+    DevBuf fb_grid, fb_Lw, fb_W, fb_picks, fb_slots, fb_ctl;
     // tuning
     int regions_override = 0;
     int force_fallback = 0;
@@ -134,6 +151,21 @@ dock_status fail(dock_ctx* c, dock_status s, const char* fmt, ...)
         if (s_ != DOCK_OK) return s_;      \
     } while (0)
 
+// 0 = host memory (pageable or pinned), 1 = device memory of `device` (or managed), -1 = device memory of
+// another device (the kernels of this context cannot use it)
+int ptr_kind(const void* p, int device)
+{
+    if (!p) return 0;
+    cudaPointerAttributes at;
+    if (cudaPointerGetAttributes(&at, p) != cudaSuccess) {
+        cudaGetLastError();
+        return 0;
+    }
+    if (at.type == cudaMemoryTypeManaged) return 1;
+    if (at.type == cudaMemoryTypeDevice) return at.device == device ? 1 : -1;
+    return 0;
+}
+
 bool is_device_ptr(const void* p)
 {
     if (!p) return false;
@@ -143,6 +175,33 @@ bool is_device_ptr(const void* p)
         return false;
     }
     return at.type == cudaMemoryTypeDevice || at.type == cudaMemoryTypeManaged;
+}
+
+// Device-or-host classification of a caller pointer; device memory of another device is an argument error.
+#define PTR_KIND(dst, p, what)                                                                           \
+    do {                                                                                                 \
+        int k_ = ptr_kind((p), ctx->device);                                                             \
+        if (k_ < 0) return fail(ctx, DOCK_E_INVALID_ARG, "%s is device memory of another device", what); \
+        dst = (k_ == 1);                                                                                 \
+    } while (0)
+
+// Next slot of the pinned staging ring (waits only for the H2D copy that last read the slot).
+dock_status acquire_stage(dock_ctx* ctx, size_t bytes, dock_ctx::Stage** out)
+{
+    dock_ctx::Stage& st = ctx->stage[ctx->stage_next];
+    ctx->stage_next = (ctx->stage_next + 1) % 3;
+    if (st.live) CU(cudaEventSynchronize(st.ev));
+    st.live = false;
+    if (bytes > st.cap) {
+        if (st.h) CU(cudaFreeHost(st.h));
+        st.h = nullptr;
+        st.cap = 0;
+        const size_t want = std::max<size_t>(bytes + bytes / 2, 1 << 16);
+        CU(cudaHostAlloc(&st.h, want, cudaHostAllocDefault));
+        st.cap = want;
+    }
+    *out = &st;
+    return DOCK_OK;
 }
 
 dock_status ensure(dock_ctx* ctx, DevBuf& b, size_t bytes)
@@ -385,34 +444,37 @@ dock_status check_ctx(dock_ctx* ctx)
 }
 
 // Stage probes (atoms packed probe by probe) and rotations on the device.
-// Returns device pointers in *xyz, *coef, *off, *rot.
+// Returns device pointers in *xyz, *coef, *off, *rot.  With fb != nullptr the fallback's per-call
+// arguments (dk::FbDyn, its vox.xyz/coef/atom_off/rot filled in here) travel in the same H2D copy and
+// *d_fb receives their device address.
 dock_status stage_inputs(dock_ctx* ctx, const dock_probe_desc* probes, int n_probes, const double* rot,
                          int n_rot, const double** d_xyz, const float** d_coef, const int** d_off,
-                         const double** d_rot)
+                         const double** d_rot, dk::FbDyn* fb = nullptr, const dk::FbDyn** d_fb = nullptr)
 {
-    // One pinned staging block [off][gather table][rot (host)][host xyz][host coef] goes up in a single
-    // H2D copy; one gather kernel then assembles all probes' atoms (device-resident probe arrays are read
-    // in place).  The host part stays short: until the first launch the GPU idles inside a timed step.
+    // One pinned staging block [fb args][off][gather table][rot (host)][host xyz][host coef] goes up in a
+    // single H2D copy; one gather kernel then assembles all probes' atoms (device-resident probe arrays are
+    // read in place).  The host part stays short and never waits for the GPU (staging ring).
     const int P = ctx->P;
     std::vector<int> off(n_probes + 1, 0);
     for (int i = 0; i < n_probes; i++) off[i + 1] = off[i] + probes[i].n_atoms;
     const int na = off[n_probes];
-    const bool rot_dev = is_device_ptr(rot);
+    bool rot_dev = false;
+    PTR_KIND(rot_dev, rot, "rot");
+    const size_t b_fb = fb ? (sizeof(dk::FbDyn) + 15) / 16 * 16 : 0;
     const size_t b_off = sizeof(int) * (n_probes + 1), b_tab = sizeof(dk::ProbeSrc) * std::max(n_probes, 1);
     const size_t b_rot = rot_dev ? 0 : sizeof(double) * 9 * n_rot;
     const size_t b_xyz = sizeof(double) * 3 * std::max(na, 1), b_coef = sizeof(float) * P * std::max(na, 1);
-    const size_t o_tab = (b_off + 15) / 16 * 16, o_rot = o_tab + (b_tab + 15) / 16 * 16;
+    const size_t o_off = b_fb, o_tab = o_off + (b_off + 15) / 16 * 16, o_rot = o_tab + (b_tab + 15) / 16 * 16;
     const size_t o_xyz = o_rot + (b_rot + 15) / 16 * 16, o_coef = o_xyz + (b_xyz + 15) / 16 * 16;
     const size_t total = o_coef + b_coef;
     TRY(ensure(ctx, ctx->xyz, b_xyz));
     TRY(ensure(ctx, ctx->coef, b_coef));
     TRY(ensure(ctx, ctx->off, total));   // device copy of the whole staging block
-    TRY(ensure_pinned(ctx, total));
-    // the previous call may still read the staging buffer
-    CU(cudaStreamSynchronize(ctx->stream));
-    char* hs = static_cast<char*>(ctx->h_stage);
+    dock_ctx::Stage* stg = nullptr;
+    TRY(acquire_stage(ctx, total, &stg));
+    char* hs = static_cast<char*>(stg->h);
     char* ds = static_cast<char*>(ctx->off.p);
-    memcpy(hs, off.data(), b_off);
+    memcpy(hs + o_off, off.data(), b_off);
     if (!rot_dev) memcpy(hs + o_rot, rot, b_rot);
     auto* tab = reinterpret_cast<dk::ProbeSrc*>(hs + o_tab);
     for (int i = 0; i < n_probes; i++) {
@@ -422,13 +484,16 @@ dock_status stage_inputs(dock_ctx* ctx, const dock_probe_desc* probes, int n_pro
         t.off = off[i];
         if (pr.n_atoms > 0) {
             const size_t bx = sizeof(double) * 3 * pr.n_atoms, bc = sizeof(float) * P * pr.n_atoms;
-            if (is_device_ptr(pr.xyz)) {
+            bool xd = false, cd = false;
+            PTR_KIND(xd, pr.xyz, "probe xyz");
+            PTR_KIND(cd, pr.coef, "probe coef");
+            if (xd) {
                 t.xyz = pr.xyz;
             } else {
                 memcpy(hs + o_xyz + sizeof(double) * 3 * (size_t)off[i], pr.xyz, bx);
                 t.xyz = reinterpret_cast<const double*>(ds + o_xyz) + 3 * (size_t)off[i];
             }
-            if (is_device_ptr(pr.coef)) {
+            if (cd) {
                 t.coef = pr.coef;
             } else {
                 memcpy(hs + o_coef + sizeof(float) * P * (size_t)off[i], pr.coef, bc);
@@ -437,7 +502,21 @@ dock_status stage_inputs(dock_ctx* ctx, const dock_probe_desc* probes, int n_pro
         }
         tab[i] = t;
     }
+    *d_rot = rot_dev ? rot : reinterpret_cast<const double*>(ds + o_rot);
+    *d_xyz = static_cast<const double*>(ctx->xyz.p);
+    *d_coef = static_cast<const float*>(ctx->coef.p);
+    *d_off = reinterpret_cast<const int*>(ds + o_off);
+    if (fb) {
+        fb->vox.xyz = *d_xyz;
+        fb->vox.coef = *d_coef;
+        fb->vox.atom_off = *d_off;
+        fb->vox.rot = *d_rot;
+        memcpy(hs, fb, sizeof(dk::FbDyn));
+        *d_fb = reinterpret_cast<const dk::FbDyn*>(ds);
+    }
     CU(cudaMemcpyAsync(ds, hs, total, cudaMemcpyHostToDevice, ctx->stream));
+    CU(cudaEventRecord(stg->ev, ctx->stream));
+    stg->live = true;
     if (n_probes > 0) {
         dk::k_gather_probes<<<n_probes, 64, 0, ctx->stream>>>(reinterpret_cast<const dk::ProbeSrc*>(ds + o_tab),
                                                               n_probes, P, static_cast<double*>(ctx->xyz.p),
@@ -445,10 +524,6 @@ dock_status stage_inputs(dock_ctx* ctx, const dock_probe_desc* probes, int n_pro
         CU(cudaGetLastError());
         ctx->kernels_last++;
     }
-    *d_rot = rot_dev ? rot : reinterpret_cast<const double*>(ds + o_rot);
-    *d_xyz = static_cast<const double*>(ctx->xyz.p);
-    *d_coef = static_cast<const float*>(ctx->coef.p);
-    *d_off = reinterpret_cast<const int*>(ds);
     return DOCK_OK;
 }
 
@@ -464,25 +539,19 @@ dock_status validate_probes(dock_ctx* ctx, const dock_probe_desc* probes, int n_
         if (p.m > ctx->m_max || p.m > DOCK_MAX_M)
             return fail(ctx, DOCK_E_UNSUPPORTED, "probe %d: m=%d exceeds m_max=%d", i, p.m, ctx->m_max);
         if (p.m != m) return fail(ctx, DOCK_E_UNSUPPORTED, "probes of different m in one batch");
-        if (!is_device_ptr(p.xyz) && p.n_atoms > 0) {
+        bool xd = false, cd = false;
+        PTR_KIND(xd, p.xyz, "probe xyz");
+        PTR_KIND(cd, p.coef, "probe coef");
+        if (!xd && p.n_atoms > 0) {
             for (int j = 0; j < 3 * p.n_atoms; j++)
                 if (!std::isfinite(p.xyz[j])) return fail(ctx, DOCK_E_INVALID_ARG, "probe %d: non-finite xyz", i);
         }
-        if (!is_device_ptr(p.coef) && p.n_atoms > 0) {
+        if (!cd && p.n_atoms > 0) {
             for (int j = 0; j < ctx->P * p.n_atoms; j++)
                 if (!std::isfinite(p.coef[j])) return fail(ctx, DOCK_E_INVALID_ARG, "probe %d: non-finite coef", i);
         }
     }
     *m_out = m;
-    return DOCK_OK;
-}
-
-dock_status check_status_word(dock_ctx* ctx)
-{
-    int st = ctx->h_small[0];
-    if (st & dk::ST_BAD_ROTATION) return fail(ctx, DOCK_E_BAD_ROTATION, "a rotation is not a proper rotation matrix");
-    if (st & dk::ST_OUTSIDE)
-        return fail(ctx, DOCK_E_PROBE_OUTSIDE_GRID, "a probe atom voxelizes outside the m^3 probe box");
     return DOCK_OK;
 }
 
@@ -541,73 +610,6 @@ dock_status run_grid(dock_ctx* ctx, int m, int n_slots, const float* Lw, float* 
     a.grid = grid;
     CU(dock_launch_ffma(m, true, ctx->plan[m].tmap, ctx->plan[m].smem, a, (int)(nb * G), ctx->stream));
     ctx->kernels_last++;
-    return DOCK_OK;
-}
-
-dock_status run_grid_tc(dock_ctx* ctx, int m, int n_slots, const float* Lw, float* grid);
-
-// Exact fallback for flagged slots: full score grid + exact greedy.  The grids come from the
-// engine that produced the candidates (use_tc: the tcgen05 GRID epilogue; else the FFMA one), so a
-// rotation's score bits never depend on whether it was flagged.
-dock_status run_fallback(dock_ctx* ctx, int m, int nfb, int64_t unit_begin, int n_rot, const double* xyz,
-                         const float* coef, const int* off, const double* rot, int k, int rho, void* poses,
-                         bool use_tc)
-{
-    std::vector<int> slots(nfb);
-    CU(cudaMemcpyAsync(slots.data(), ctx->fb_list.p, sizeof(int) * nfb, cudaMemcpyDeviceToHost, ctx->stream));
-    CU(cudaStreamSynchronize(ctx->stream));
-    std::sort(slots.begin(), slots.end());
-    const size_t ncell = (size_t)ctx->nx * ctx->ny * ctx->nz;
-    const int chunk = (int)std::max<size_t>(1, std::min<size_t>(32, (size_t(1) << 30) / (ncell * 4)));
-    TRY(ensure(ctx, ctx->grid, sizeof(float) * ncell * chunk));
-    TRY(ensure(ctx, ctx->slots, sizeof(int) * 2 * chunk));
-    TRY(ensure(ctx, ctx->picks, sizeof(unsigned long long) * chunk * k));
-    const int m3 = m * m * m;
-    TRY(ensure(ctx, ctx->Lw_fb, sizeof(float) * ((chunk + dk::RB - 1) / dk::RB) * dk::RB * ctx->P * m3));
-    TRY(ensure_pinned(ctx, sizeof(int) * 2 * chunk));
-    for (int c0 = 0; c0 < nfb; c0 += chunk) {
-        int n = std::min(chunk, nfb - c0);
-        CU(cudaStreamSynchronize(ctx->stream));
-        int* h = static_cast<int*>(ctx->h_stage);
-        for (int i = 0; i < n; i++) {
-            h[i] = (int)(unit_begin + slots[c0 + i]);   // absolute unit
-            h[chunk + i] = slots[c0 + i];                // output slot
-        }
-        CU(cudaMemcpyAsync(ctx->slots.p, h, sizeof(int) * 2 * chunk, cudaMemcpyHostToDevice, ctx->stream));
-        const int* d_units = static_cast<const int*>(ctx->slots.p);
-        const int* d_outslot = d_units + chunk;
-        TRY(run_voxelize(ctx, m, n, 0, d_units, n_rot, xyz, coef, off, rot, ctx->d_w,
-                         static_cast<float*>(ctx->Lw_fb.p)));
-        if (use_tc)
-            TRY(run_grid_tc(ctx, m, n, static_cast<const float*>(ctx->Lw_fb.p), static_cast<float*>(ctx->grid.p)));
-        else
-            TRY(run_grid(ctx, m, n, static_cast<const float*>(ctx->Lw_fb.p), static_cast<float*>(ctx->grid.p)));
-        dk::GreedyArgs ga{};
-        ga.grid = static_cast<const float*>(ctx->grid.p);
-        ga.slots = d_outslot;
-        ga.picks = static_cast<unsigned long long*>(ctx->picks.p);
-        ga.n = n;
-        ga.k = k;
-        ga.rho = rho;
-        ga.n_rot = n_rot;
-        ga.nx = ctx->nx;
-        ga.ny = ctx->ny;
-        ga.nz = ctx->nz;
-        ga.unit_begin = unit_begin;
-        ga.poses = poses;
-        ga.flag_bits = 1u;   // DOCK_POSE_FALLBACK
-        dk::k_fill_u64<<<1, 256, 0, ctx->stream>>>(ga.picks, (size_t)n * k, dk::KEY_MAX);
-        CU(cudaGetLastError());
-        const int per_grid = std::max(8, std::min(512, 16 * ctx->n_sms / std::max(1, n)));
-        for (int j = 0; j < k; j++) {
-            ga.round = j;
-            dk::k_greedy_round<<<n * per_grid, 256, 0, ctx->stream>>>(ga);
-            CU(cudaGetLastError());
-        }
-        dk::k_greedy_emit<<<(n * k + 127) / 128, 128, 0, ctx->stream>>>(ga);
-        CU(cudaGetLastError());
-        ctx->kernels_last += k + 2;
-    }
     return DOCK_OK;
 }
 
@@ -670,14 +672,15 @@ dock_status select_engine(dock_ctx* ctx, int m, bool* use_tc)
 }
 
 // Pack folded FP32 weights into the tcgen05 A-operand layout of variant v.
-dock_status pack_weights_tc(dock_ctx* ctx, int m, int v, int n_slots, const float* Lw)
+dock_status pack_weights_tc(dock_ctx* ctx, int m, int v, int n_slots, const float* Lw, DevBuf* dst = nullptr)
 {
     const TcPlan& tp = ctx->tcplan[v][m];
     const int64_t n_blocks = (n_slots + tc::ROT - 1) / tc::ROT;
-    TRY(ensure(ctx, ctx->Wtc, (size_t)n_blocks * tp.nsteps * tc::WCHUNK));
+    DevBuf& Wb = dst ? *dst : ctx->Wtc;
+    TRY(ensure(ctx, Wb, (size_t)n_blocks * tp.nsteps * tc::WCHUNK));
     const int64_t rows = n_blocks * tp.nsteps * 2 * tc::ROT;
     const int grid = (int)std::min<int64_t>((rows + 255) / 256, 65535);
-    unsigned char* W = static_cast<unsigned char*>(ctx->Wtc.p);
+    unsigned char* W = static_cast<unsigned char*>(Wb.p);
     if (v == 1)
         tc::k_pack_weights_tc_pair<<<grid, 256, 0, ctx->stream>>>(Lw, W, n_slots, ctx->P, m, tp.S1, tp.S1p, tp.S2,
                                                                    tp.S2p);
@@ -761,6 +764,251 @@ dock_status run_grid_tc(dock_ctx* ctx, int m, int n_slots, const float* Lw, floa
     return DOCK_OK;
 }
 
+// ---------------------------------------------------------------- device-driven exact fallback
+//
+// Rotations k_merge flagged (candidate overflow, or a list whose last key is below the last pick; DESIGN.md
+// §8) get their full score grid from the engine that produced their candidates (tcgen05 GRID epilogue or
+// FFMA GRID epilogue: identical score bits) and the exact best-then-exclude greedy.  The
+// number of flagged rotations is only known on the device, so the fallback is one CUDA graph:
+//   k_fb_init (condition = fb_cnt > 0) -> WHILE { k_fb_chunk -> k_voxelize_dyn -> [pack] -> GRID correlation
+//   -> k_fill_u64 -> k rounds k_greedy_round -> k_greedy_emit -> k_fb_advance (condition = more left) }
+// over chunks of `ch` flagged slots.  Every per-call value (poses, unit_begin, n_rot, input pointers) is
+// read from the dk::FbDyn block uploaded with the call's inputs, so the instantiated graph is reused
+// across calls with the same shape; the host never waits for the flag count.
+
+struct FbKey {   // everything the captured fallback graph bakes in (compared bytewise)
+    int m, use_tc, v, G, k, rho, ch, nepi, P, nx, ny, nz;
+    const void *fb_list, *d_small, *dyn, *grid, *Lw, *W, *picks, *slots, *ctl, *w;
+};
+static_assert(sizeof(FbKey) <= sizeof(((dock_ctx*)nullptr)->fb_key), "fb_key too small");
+
+int fb_chunk(const dock_ctx* ctx, bool use_tc)
+{
+    const size_t ncell = (size_t)ctx->nx * ctx->ny * ctx->nz;
+    const size_t budget = size_t(1) << 30;   // score grids of one chunk: <= 1 GiB
+    const size_t fit = std::max<size_t>(1, budget / (ncell * sizeof(float)));
+    return (int)std::min<size_t>(use_tc ? tc::ROT : 64, fit);
+}
+
+dock_status fb_buffers(dock_ctx* ctx, int m, int ch, int k)
+{
+    const size_t ncell = (size_t)ctx->nx * ctx->ny * ctx->nz;
+    const int m3 = m * m * m;
+    TRY(ensure(ctx, ctx->fb_grid, sizeof(float) * ncell * ch));
+    TRY(ensure(ctx, ctx->fb_Lw, sizeof(float) * ((ch + dk::RB - 1) / dk::RB) * dk::RB * ctx->P * m3));
+    TRY(ensure(ctx, ctx->fb_picks, sizeof(unsigned long long) * ch * k));
+    TRY(ensure(ctx, ctx->fb_slots, sizeof(int) * ch));
+    TRY(ensure(ctx, ctx->fb_ctl, sizeof(dk::FbCtl)));
+    return DOCK_OK;
+}
+
+// Capture + instantiate the fallback graph for this key (ctx->stream is redirected to the private capture
+// streams while the existing launch helpers record into the graph).
+dock_status build_fb_graph(dock_ctx* ctx, const FbKey& key, const dk::FbDyn* d_dyn)
+{
+    if (ctx->fb_exec) {
+        cudaGraphExecDestroy(ctx->fb_exec);
+        ctx->fb_exec = nullptr;
+    }
+    const int m = key.m, ch = key.ch, k = key.k;
+    auto* fb_cnt = reinterpret_cast<unsigned int*>(ctx->d_small + 1);
+    auto* ctl = static_cast<dk::FbCtl*>(ctx->fb_ctl.p);
+    int* slots = static_cast<int*>(ctx->fb_slots.p);
+    cudaStream_t user = ctx->stream, cs = ctx->cap_stream, cs2 = ctx->cap_stream2;
+    cudaGraph_t graph = nullptr;
+    dock_status st = DOCK_OK;
+    auto body = [&]() -> dock_status {
+        CU(cudaStreamBeginCapture(cs, cudaStreamCaptureModeThreadLocal));
+        cudaStreamCaptureStatus cst;
+        cudaGraph_t g = nullptr;
+        const cudaGraphNode_t* deps = nullptr;
+        size_t nd = 0;
+        CU(cudaStreamGetCaptureInfo(cs, &cst, nullptr, &g, &deps, &nd));
+        cudaGraphConditionalHandle h;
+        CU(cudaGraphConditionalHandleCreate(&h, g, 0, 0));
+        dk::k_fb_init<<<1, 1, 0, cs>>>(h, fb_cnt, ctl);
+        CU(cudaGetLastError());
+        CU(cudaStreamGetCaptureInfo(cs, &cst, nullptr, &g, &deps, &nd));
+        cudaGraphNodeParams cp = {};
+        cp.type = cudaGraphNodeTypeConditional;
+        cp.conditional.handle = h;
+        cp.conditional.type = cudaGraphCondTypeWhile;
+        cp.conditional.size = 1;
+        cudaGraphNode_t node;
+        CU(cudaGraphAddNode(&node, g, deps, nd, &cp));
+        cudaGraph_t loop = cp.conditional.phGraph_out[0];
+        CU(cudaStreamUpdateCaptureDependencies(cs, &node, 1, cudaStreamSetCaptureDependencies));
+        // loop body, captured on the second private stream
+        CU(cudaStreamBeginCaptureToGraph(cs2, loop, nullptr, nullptr, 0, cudaStreamCaptureModeThreadLocal));
+        ctx->stream = cs2;
+        dk::k_fb_chunk<<<1, 128, 0, cs2>>>(fb_cnt, static_cast<const int*>(ctx->fb_list.p), ctl, slots, ch);
+        CU(cudaGetLastError());
+        const int nvox = (ch + dk::RB - 1) / dk::RB * dk::RB * ctx->P;
+        dk::k_voxelize_dyn<<<(nvox + 127) / 128, 128, 0, cs2>>>(&d_dyn->vox);
+        CU(cudaGetLastError());
+        const float* Lw = static_cast<const float*>(ctx->fb_Lw.p);
+        float* grid = static_cast<float*>(ctx->fb_grid.p);
+        if (key.use_tc) {
+            TRY(pack_weights_tc(ctx, m, key.v, ch, Lw, &ctx->fb_W));
+            tc::TcArgs a = tc_args(ctx, m, key.v, ch, key.G, static_cast<const unsigned char*>(ctx->fb_W.p));
+            a.grid = grid;
+            a.n_live = &ctl->n_live;
+            a.trace = nullptr;
+            CU(launch_tc(m, key.v, true, ctx->tcplan[key.v][m], a, key.G, cs2));
+        } else {
+            const int64_t nb = (ch + dk::RB - 1) / dk::RB;
+            dk::CorrArgs a = corr_args(ctx, m, ch, key.G, Lw);
+            a.grid = grid;
+            a.n_live = &ctl->n_live;
+            CU(dock_launch_ffma(m, true, ctx->plan[m].tmap, ctx->plan[m].smem, a, (int)(nb * key.G), cs2));
+        }
+        dk::GreedyArgs ga{};
+        ga.grid = grid;
+        ga.slots = slots;
+        ga.picks = static_cast<unsigned long long*>(ctx->fb_picks.p);
+        ga.n = ch;
+        ga.k = k;
+        ga.rho = key.rho;
+        ga.nx = ctx->nx;
+        ga.ny = ctx->ny;
+        ga.nz = ctx->nz;
+        ga.flag_bits = 1u;   // DOCK_POSE_FALLBACK
+        ga.n_live = &ctl->n_live;
+        ga.dyn = d_dyn;
+        dk::k_fill_u64<<<1, 256, 0, cs2>>>(ga.picks, (size_t)ch * k, dk::KEY_MAX);
+        CU(cudaGetLastError());
+        const int per_grid = std::max(8, std::min(512, 16 * ctx->n_sms / std::max(1, ch)));
+        for (int j = 0; j < k; j++) {
+            ga.round = j;
+            dk::k_greedy_round<<<ch * per_grid, 256, 0, cs2>>>(ga);
+            CU(cudaGetLastError());
+        }
+        dk::k_greedy_emit<<<(ch * k + 127) / 128, 128, 0, cs2>>>(ga);
+        CU(cudaGetLastError());
+        dk::k_fb_advance<<<1, 1, 0, cs2>>>(h, fb_cnt, ctl, ch);
+        CU(cudaGetLastError());
+        ctx->stream = user;
+        CU(cudaStreamEndCapture(cs2, nullptr));
+        CU(cudaStreamEndCapture(cs, &graph));
+        CU(cudaGraphInstantiate(&ctx->fb_exec, graph, 0));
+        return DOCK_OK;
+    };
+    st = body();
+    ctx->stream = user;
+    if (st != DOCK_OK) {   // leave no capture open on the private streams
+        cudaGraph_t junk = nullptr;
+        cudaStreamCaptureStatus cst;
+        if (cudaStreamIsCapturing(cs2, &cst) == cudaSuccess && cst != cudaStreamCaptureStatusNone)
+            cudaStreamEndCapture(cs2, &junk);
+        if (cudaStreamIsCapturing(cs, &cst) == cudaSuccess && cst != cudaStreamCaptureStatusNone)
+            cudaStreamEndCapture(cs, &junk);
+        if (junk) cudaGraphDestroy(junk);
+        cudaGetLastError();
+        memset(ctx->fb_key, 0, sizeof(ctx->fb_key));
+    }
+    if (graph) cudaGraphDestroy(graph);
+    return st;
+}
+
+// Enqueue the fallback graph on the context stream (no host synchronisation).
+dock_status launch_fallback(dock_ctx* ctx, int m, bool use_tc, int v, int k, int rho, const dk::FbDyn* d_dyn)
+{
+    const int ch = fb_chunk(ctx, use_tc);
+    TRY(fb_buffers(ctx, m, ch, k));
+    FbKey key;
+    memset(&key, 0, sizeof(key));
+    key.m = m;
+    key.use_tc = use_tc;
+    key.v = use_tc ? v : 0;
+    if (use_tc) {
+        int vv = 0, G = 0;
+        if (!plan_tc_launch(ctx, m, ch, &vv, &G)) return fail(ctx, DOCK_E_UNSUPPORTED, "no tensor-core plan");
+        key.v = vv;
+        key.G = G;
+        const TcPlan& tp = ctx->tcplan[vv][m];
+        TRY(ensure(ctx, ctx->fb_W, (size_t)tp.nsteps * tc::WCHUNK));
+    } else {
+        key.G = choose_regions(ctx, (ch + dk::RB - 1) / dk::RB);
+    }
+    key.k = k;
+    key.rho = rho;
+    key.ch = ch;
+    key.nepi = ctx->tc_nepi;
+    key.P = ctx->P;
+    key.nx = ctx->nx;
+    key.ny = ctx->ny;
+    key.nz = ctx->nz;
+    key.fb_list = ctx->fb_list.p;
+    key.d_small = ctx->d_small;
+    key.dyn = d_dyn;
+    key.grid = ctx->fb_grid.p;
+    key.Lw = ctx->fb_Lw.p;
+    key.W = ctx->fb_W.p;
+    key.picks = ctx->fb_picks.p;
+    key.slots = ctx->fb_slots.p;
+    key.ctl = ctx->fb_ctl.p;
+    key.w = ctx->d_w;
+    if (!ctx->fb_exec || memcmp(&key, ctx->fb_key, sizeof(key)) != 0) {
+        TRY(build_fb_graph(ctx, key, d_dyn));
+        memcpy(ctx->fb_key, &key, sizeof(key));
+    }
+    CU(cudaGraphLaunch(ctx->fb_exec, ctx->stream));
+    ctx->kernels_last++;   // k_fb_init; the loop body runs only for flagged rotations
+    return DOCK_OK;
+}
+
+// Template of the per-call fallback arguments (the input pointers are filled by stage_inputs).
+dk::FbDyn fb_template(dock_ctx* ctx, int m, int ch, int64_t unit_begin, int n_rot, void* poses)
+{
+    dk::FbDyn f;
+    memset(&f, 0, sizeof(f));
+    f.vox.w = ctx->d_w;
+    f.vox.unit_list = static_cast<const int*>(ctx->fb_slots.p);
+    f.vox.unit_begin = unit_begin;
+    f.vox.n_rot = n_rot;
+    f.vox.n_slots = ch;
+    f.vox.P = ctx->P;
+    f.vox.m = m;
+    f.vox.spacing = ctx->spacing;
+    f.vox.Lw = static_cast<float*>(ctx->fb_Lw.p);
+    f.vox.status = ctx->d_small;
+    f.vox.n_live = &static_cast<dk::FbCtl*>(ctx->fb_ctl.p)->n_live;
+    f.poses = poses;
+    f.unit_begin = unit_begin;
+    f.n_rot = n_rot;
+    return f;
+}
+
+// Queue the copy of the status words for the next sync point (asynchronous).
+dock_status end_call(dock_ctx* ctx)
+{
+    CU(cudaMemcpyAsync(ctx->h_small, ctx->d_small, 16, cudaMemcpyDeviceToHost, ctx->stream));
+    CU(cudaEventRecord(ctx->ev_done, ctx->stream));
+    ctx->unsynced = true;
+    return DOCK_OK;
+}
+
+// Sync point: wait for the context stream, take the stats of the last call and report (then clear) the
+// sticky device status bits of every call since the previous sync point.
+dock_status sync_point(dock_ctx* ctx)
+{
+    CU(cudaStreamSynchronize(ctx->stream));
+    ctx->unsynced = false;
+    ctx->fallback_last = (unsigned)ctx->h_small[1];
+    ctx->cand_max_last = (unsigned)ctx->h_small[2];
+    const int st = ctx->h_small[0];
+    if (st) {
+        ctx->h_small[0] = 0;
+        CU(cudaMemsetAsync(ctx->d_small, 0, 4, ctx->stream));
+        CU(cudaStreamSynchronize(ctx->stream));
+        if (st & dk::ST_BAD_ROTATION)
+            return fail(ctx, DOCK_E_BAD_ROTATION, "a rotation is not a proper rotation matrix");
+        if (st & dk::ST_OUTSIDE)
+            return fail(ctx, DOCK_E_PROBE_OUTSIDE_GRID, "a probe atom voxelizes outside the m^3 probe box");
+    }
+    return DOCK_OK;
+}
+
 }  // namespace
 
 // =====================================================================================  ABI
@@ -788,8 +1036,10 @@ void dock_destroy(dock_ctx* ctx)
     if (!ctx) return;
     cudaSetDevice(ctx->device);
     if (ctx->stream) cudaStreamSynchronize(ctx->stream);
-    DevBuf* bufs[] = {&ctx->xyz, &ctx->coef, &ctx->off, &ctx->rot, &ctx->Lw, &ctx->T, &ctx->mu, &ctx->cnt,
-                      &ctx->cand, &ctx->poses, &ctx->fb_list, &ctx->grid, &ctx->slots, &ctx->units, &ctx->Lw_fb, &ctx->picks};
+    DevBuf* bufs[] = {&ctx->xyz,     &ctx->coef,     &ctx->off,    &ctx->rot,      &ctx->Lw,       &ctx->T,
+                      &ctx->mu,      &ctx->cnt,      &ctx->cand,   &ctx->poses,    &ctx->fb_list,  &ctx->grid,
+                      &ctx->slots,   &ctx->units,    &ctx->Lw_fb,  &ctx->picks,    &ctx->fb_grid,  &ctx->fb_Lw,
+                      &ctx->fb_W,    &ctx->fb_picks, &ctx->fb_slots, &ctx->fb_ctl};
     for (DevBuf* b : bufs)
         if (b->p) cudaFree(b->p);
     if (ctx->d_trace) cudaFree(ctx->d_trace);
@@ -804,6 +1054,14 @@ void dock_destroy(dock_ctx* ctx)
     if (ctx->d_small) cudaFree(ctx->d_small);
     if (ctx->h_small) cudaFreeHost(ctx->h_small);
     if (ctx->h_stage) cudaFreeHost(ctx->h_stage);
+    for (auto& st : ctx->stage) {
+        if (st.h) cudaFreeHost(st.h);
+        if (st.ev) cudaEventDestroy(st.ev);
+    }
+    if (ctx->fb_exec) cudaGraphExecDestroy(ctx->fb_exec);
+    if (ctx->ev_done) cudaEventDestroy(ctx->ev_done);
+    if (ctx->cap_stream) cudaStreamDestroy(ctx->cap_stream);
+    if (ctx->cap_stream2) cudaStreamDestroy(ctx->cap_stream2);
     for (cudaEvent_t e : ctx->ev_corr)
         if (e) cudaEventDestroy(e);
     if (ctx->own_stream && ctx->stream) cudaStreamDestroy(ctx->stream);
@@ -845,8 +1103,13 @@ dock_status dock_init(const dock_grid_desc* g, const float* receptor, const floa
         if (cudaStreamCreateWithFlags(&ctx->stream, cudaStreamNonBlocking) != cudaSuccess) return bail(DOCK_E_CUDA);
         ctx->own_stream = true;
     }
-    if (cudaEventCreate(&ctx->ev_corr[0]) != cudaSuccess || cudaEventCreate(&ctx->ev_corr[1]) != cudaSuccess)
+    if (cudaEventCreate(&ctx->ev_corr[0]) != cudaSuccess || cudaEventCreate(&ctx->ev_corr[1]) != cudaSuccess ||
+        cudaEventCreateWithFlags(&ctx->ev_done, cudaEventDisableTiming) != cudaSuccess ||
+        cudaStreamCreateWithFlags(&ctx->cap_stream, cudaStreamNonBlocking) != cudaSuccess ||
+        cudaStreamCreateWithFlags(&ctx->cap_stream2, cudaStreamNonBlocking) != cudaSuccess)
         return bail(DOCK_E_CUDA);
+    for (auto& st : ctx->stage)
+        if (cudaEventCreateWithFlags(&st.ev, cudaEventDisableTiming) != cudaSuccess) return bail(DOCK_E_CUDA);
     if (const char* e = getenv("DOCK_TC_DEBUG")) ctx->tc_dbg = atoi(e);
     if (const char* e = getenv("DOCK_TC_TRACE")) {
         if (atoi(e) > 0 && cudaMalloc(&ctx->d_trace, sizeof(unsigned long long) * tc::TR_N) != cudaSuccess)
@@ -863,7 +1126,9 @@ dock_status dock_init(const dock_grid_desc* g, const float* receptor, const floa
 
     // weights (host or device) -> host copy for validation
     std::vector<float> w(P);
-    if (is_device_ptr(weights)) {
+    const int wk = ptr_kind(weights, ctx->device), rk = ptr_kind(receptor, ctx->device);
+    if (wk < 0 || rk < 0) return bail(DOCK_E_INVALID_ARG);   // device memory of another device
+    if (wk == 1) {
         if (cudaMemcpy(w.data(), weights, sizeof(float) * P, cudaMemcpyDeviceToHost) != cudaSuccess)
             return bail(DOCK_E_CUDA);
     } else {
@@ -877,7 +1142,7 @@ dock_status dock_init(const dock_grid_desc* g, const float* receptor, const floa
         return bail(DOCK_E_OOM);
     }
     float* d_src = nullptr;
-    bool rec_dev = is_device_ptr(receptor);
+    bool rec_dev = rk == 1;
     if (rec_dev) {
         d_src = const_cast<float*>(receptor);
     } else {
@@ -1034,6 +1299,15 @@ dock_status dock_get_info(const dock_ctx* ctx, dock_info* info)
         info->tc_row_last = tp.ntt;
         info->tc_rows_per_tile_last = tp.q;
     }
+    info->pending = ctx->unsynced ? 1 : 0;
+    if (ctx->unsynced && ctx->ev_done && cudaEventQuery(ctx->ev_done) == cudaSuccess) {
+        // the last call has completed: its statistics are readable without a sync point
+        info->pending = 0;
+        info->fallback_last = (unsigned)ctx->h_small[1];
+        info->cand_max_last = (unsigned)ctx->h_small[2];
+    }
+    cudaGetLastError();
+    info->fb_chunk = fb_chunk(ctx, ctx->engine_last == 2);
     return DOCK_OK;
 }
 
@@ -1056,21 +1330,19 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
     if (unit_begin < 0 || unit_end < unit_begin || unit_end > (int64_t)n_probes * n_rot)
         return fail(ctx, DOCK_E_INVALID_ARG, "bad unit range");
     const int64_t n_units64 = unit_end - unit_begin;
-    if (n_units64 > (int64_t)1 << 28) return fail(ctx, DOCK_E_UNSUPPORTED, "too many units in one call");
+    // 32-bit index math of the per-call kernels: (units rounded to RB) * P must fit in an int
+    if (n_units64 > (int64_t)1 << 28 || (n_units64 + dk::RB) * ctx->P > 0x7fffffffLL)
+        return fail(ctx, DOCK_E_UNSUPPORTED, "too many units in one call");
     const int n_units = (int)n_units64;
-    if (n_units == 0) return DOCK_OK;
+    bool out_dev = false, rot_dev = false;
+    PTR_KIND(out_dev, out, "out");
+    PTR_KIND(rot_dev, rot, "rot");
+    if (n_units == 0) return out_dev ? DOCK_OK : sync_point(ctx);
     TRY(make_plan(ctx, m));
-
-    const bool rot_dev = is_device_ptr(rot);
     if (!rot_dev) {
         for (int64_t i = 0; i < (int64_t)9 * n_rot; i++)
             if (!std::isfinite(rot[i])) return fail(ctx, DOCK_E_INVALID_ARG, "non-finite rotation");
     }
-    const double *d_xyz, *d_rot;
-    const float* d_coef;
-    const int* d_off;
-    TRY(stage_inputs(ctx, probes, n_probes, rot, n_rot, &d_xyz, &d_coef, &d_off, &d_rot));
-
     const int P = ctx->P, m3 = m * m * m;
     const int64_t n_batches = (n_units + dk::RB - 1) / dk::RB;
     const int cap = ctx->cand_cap;
@@ -1080,56 +1352,63 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
     TRY(ensure(ctx, ctx->cnt, sizeof(unsigned int) * n_units));
     TRY(ensure(ctx, ctx->cand, sizeof(unsigned long long) * (size_t)n_units * cap));
     TRY(ensure(ctx, ctx->fb_list, sizeof(int) * n_units));
-    const bool out_dev = is_device_ptr(out);
     void* d_poses = out;
     if (!out_dev) {
         TRY(ensure(ctx, ctx->poses, sizeof(dock_pose) * (size_t)n_units * k));
         d_poses = ctx->poses.p;
     }
+    // the direct engines' fallback buffers exist before staging (their addresses travel in dk::FbDyn)
+    bool use_tc = false;
+    if (ctx->engine != 3) {
+        TRY(select_engine(ctx, m, &use_tc));
+        TRY(fb_buffers(ctx, m, fb_chunk(ctx, use_tc), k));
+    }
+    dk::FbDyn fb = fb_template(ctx, m, fb_chunk(ctx, use_tc), unit_begin, n_rot, d_poses);
+    const double *d_xyz, *d_rot;
+    const float* d_coef;
+    const int* d_off;
+    const dk::FbDyn* d_fb = nullptr;
+    TRY(stage_inputs(ctx, probes, n_probes, rot, n_rot, &d_xyz, &d_coef, &d_off, &d_rot, &fb, &d_fb));
 
     unsigned int* fb_cnt = reinterpret_cast<unsigned int*>(ctx->d_small + 1);
     unsigned int* cand_max = reinterpret_cast<unsigned int*>(ctx->d_small + 2);
-    CU(cudaMemsetAsync(ctx->d_small, 0, 4, ctx->stream));
     dk::k_reset<<<(n_units + 255) / 256, 256, 0, ctx->stream>>>(
         static_cast<unsigned long long*>(ctx->T.p), static_cast<unsigned long long*>(ctx->mu.p),
         static_cast<unsigned int*>(ctx->cnt.p), n_units, fb_cnt, cand_max);
     CU(cudaGetLastError());
     ctx->kernels_last++;
 
-    // a1: voxelize (+ rotation / box validation)
+    // a1: voxelize (+ rotation / box validation; errors are sticky device status bits)
     TRY(run_voxelize(ctx, m, n_units, unit_begin, nullptr, n_rot, d_xyz, d_coef, d_off, d_rot, ctx->d_w,
                      static_cast<float*>(ctx->Lw.p)));
 
     if (ctx->engine == 3) {
-        // comparison engine: FFT score grids + exact greedy (no fused top-k, no fallback needed)
+        // comparison engine: FFT score grids + exact greedy (no fused top-k, no fallback needed); this engine
+        // synchronises internally (host-driven chunking), whatever the output memory
         ctx->engine_last = 3;
         ctx->tc_variant_last = 0;
         CU(cudaEventRecord(ctx->ev_corr[0], ctx->stream));
         TRY(run_fft_poses(ctx, m, n_units, unit_begin, n_rot, k, rho, d_poses));
         CU(cudaEventRecord(ctx->ev_corr[1], ctx->stream));
         ctx->ev_corr_valid = true;
-        ctx->fallback_last = 0;
-        CU(cudaMemcpyAsync(ctx->h_small, ctx->d_small, 16, cudaMemcpyDeviceToHost, ctx->stream));
-        CU(cudaStreamSynchronize(ctx->stream));
-        TRY(check_status_word(ctx));
         if (!out_dev)
             CU(cudaMemcpyAsync(out, d_poses, sizeof(dock_pose) * (size_t)n_units * k, cudaMemcpyDeviceToHost,
                                ctx->stream));
-        CU(cudaStreamSynchronize(ctx->stream));
-        return DOCK_OK;
+        TRY(end_call(ctx));
+        return sync_point(ctx);
     }
 
     // a2-a5: correlation + fused weighted score + on-chip top-k lists (no score grid in HBM)
-    bool use_tc = false;
-    TRY(select_engine(ctx, m, &use_tc));
     auto* Tp = static_cast<unsigned long long*>(ctx->T.p);
     auto* mup = static_cast<unsigned long long*>(ctx->mu.p);
     auto* cntp = static_cast<unsigned int*>(ctx->cnt.p);
     auto* candp = static_cast<unsigned long long*>(ctx->cand.p);
+    int v_used = 0;
     if (use_tc) {
         const int64_t n_blocks = (n_units + tc::ROT - 1) / tc::ROT;
         int v = 0, G = 0;
         if (!plan_tc_launch(ctx, m, n_units, &v, &G)) return fail(ctx, DOCK_E_UNSUPPORTED, "no tensor-core plan");
+        v_used = v;
         TRY(pack_weights_tc(ctx, m, v, n_units, static_cast<const float*>(ctx->Lw.p)));
         ctx->tc_variant_last = v;
         ctx->tc_ksteps_last = ctx->tcplan[v][m].nsteps;
@@ -1211,19 +1490,22 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
     CU(cudaGetLastError());
     ctx->kernels_last++;
 
-    CU(cudaMemcpyAsync(ctx->h_small, ctx->d_small, 16, cudaMemcpyDeviceToHost, ctx->stream));
-    CU(cudaStreamSynchronize(ctx->stream));
-    TRY(check_status_word(ctx));
-    const int nfb = ctx->h_small[1];
-    ctx->fallback_last = nfb;
-    ctx->cand_max_last = (unsigned)ctx->h_small[2];
-    if (nfb > 0)
-        TRY(run_fallback(ctx, m, nfb, unit_begin, n_rot, d_xyz, d_coef, d_off, d_rot, k, rho, d_poses, use_tc));
+    // a6': exact fallback of the flagged rotations, driven by the device-side flag count
+    TRY(launch_fallback(ctx, m, use_tc, v_used, k, rho, d_fb));
+
+    // a7: output.  Device output: return now (results and errors at dock_sync / the next sync point);
+    // host output: copy back and synchronise.
     if (!out_dev)
         CU(cudaMemcpyAsync(out, d_poses, sizeof(dock_pose) * (size_t)n_units * k, cudaMemcpyDeviceToHost,
                            ctx->stream));
-    CU(cudaStreamSynchronize(ctx->stream));
-    return DOCK_OK;
+    TRY(end_call(ctx));
+    return out_dev ? DOCK_OK : sync_point(ctx);
+}
+
+dock_status dock_sync(dock_ctx* ctx)
+{
+    TRY(check_ctx(ctx));
+    return sync_point(ctx);
 }
 
 dock_status dock_probe(dock_ctx* ctx, const dock_probe_desc* probe, const double* rot, int n_rot, int k, int rho,
@@ -1248,13 +1530,13 @@ dock_status dock_score_grid(dock_ctx* ctx, const dock_probe_desc* probe, const d
     const size_t ncell = (size_t)ctx->nx * ctx->ny * ctx->nz;
     const int m3 = m * m * m;
     TRY(ensure(ctx, ctx->Lw, sizeof(float) * ctx->P * m3 * dk::RB));
-    const bool out_dev = is_device_ptr(out);
-    const bool pt_dev = per_term && is_device_ptr(per_term);
+    bool out_dev = false, pt_dev = false;
+    PTR_KIND(out_dev, out, "out");
+    PTR_KIND(pt_dev, per_term, "per_term");
     size_t need = (out_dev ? 0 : ncell) + (per_term && !pt_dev ? ncell * ctx->P : 0);
     if (need) TRY(ensure(ctx, ctx->grid, sizeof(float) * need));
     float* g_out = out_dev ? out : static_cast<float*>(ctx->grid.p);
     float* g_pt = per_term ? (pt_dev ? per_term : static_cast<float*>(ctx->grid.p) + (out_dev ? 0 : ncell)) : nullptr;
-    CU(cudaMemsetAsync(ctx->d_small, 0, 4, ctx->stream));
     bool use_tc = false;
     if (ctx->engine == 3) ctx->engine_last = 3;
     else TRY(select_engine(ctx, m, &use_tc));
@@ -1272,14 +1554,11 @@ dock_status dock_score_grid(dock_ctx* ctx, const dock_probe_desc* probe, const d
             TRY(grid_fn(g_pt + ncell * p));
         }
     }
-    CU(cudaMemcpyAsync(ctx->h_small, ctx->d_small, 16, cudaMemcpyDeviceToHost, ctx->stream));
-    CU(cudaStreamSynchronize(ctx->stream));
-    TRY(check_status_word(ctx));
     if (!out_dev) CU(cudaMemcpyAsync(out, g_out, sizeof(float) * ncell, cudaMemcpyDeviceToHost, ctx->stream));
     if (per_term && !pt_dev)
         CU(cudaMemcpyAsync(per_term, g_pt, sizeof(float) * ncell * ctx->P, cudaMemcpyDeviceToHost, ctx->stream));
-    CU(cudaStreamSynchronize(ctx->stream));
-    return DOCK_OK;
+    TRY(end_call(ctx));
+    return sync_point(ctx);
 }
 
 dock_status dock_voxelize(dock_ctx* ctx, const dock_probe_desc* probe, const double* rot, int n_rot, float* out)
@@ -1297,23 +1576,22 @@ dock_status dock_voxelize(dock_ctx* ctx, const dock_probe_desc* probe, const dou
     const int m3 = m * m * m, P = ctx->P;
     const int64_t nb = (n_rot + dk::RB - 1) / dk::RB;
     TRY(ensure(ctx, ctx->Lw, sizeof(float) * nb * P * m3 * dk::RB));
-    const bool out_dev = is_device_ptr(out);
+    bool out_dev = false;
+    PTR_KIND(out_dev, out, "out");
     const size_t n_out = (size_t)n_rot * P * m3;
+    if ((int64_t)n_rot * P * m3 + (int64_t)dk::RB * P * m3 > 0x7fffffffLL)
+        return fail(ctx, DOCK_E_UNSUPPORTED, "too many rotations in one call");
     if (!out_dev) TRY(ensure(ctx, ctx->grid, sizeof(float) * n_out));
     float* g_out = out_dev ? out : static_cast<float*>(ctx->grid.p);
-    CU(cudaMemsetAsync(ctx->d_small, 0, 4, ctx->stream));
     TRY(run_voxelize(ctx, m, n_rot, 0, nullptr, n_rot, d_xyz, d_coef, d_off, d_rot, ctx->d_ones,
                      static_cast<float*>(ctx->Lw.p)));
     int n = (int)n_out;
     dk::k_unpack_L<<<(n + 255) / 256, 256, 0, ctx->stream>>>(static_cast<const float*>(ctx->Lw.p), g_out, n_rot, P,
                                                               m3);
     CU(cudaGetLastError());
-    CU(cudaMemcpyAsync(ctx->h_small, ctx->d_small, 16, cudaMemcpyDeviceToHost, ctx->stream));
-    CU(cudaStreamSynchronize(ctx->stream));
-    TRY(check_status_word(ctx));
     if (!out_dev) CU(cudaMemcpyAsync(out, g_out, sizeof(float) * n_out, cudaMemcpyDeviceToHost, ctx->stream));
-    CU(cudaStreamSynchronize(ctx->stream));
-    return DOCK_OK;
+    TRY(end_call(ctx));
+    return sync_point(ctx);
 }
 
 }  // extern "C"

@@ -59,6 +59,7 @@ struct CorrArgs {
     int cap;
     // grid mode
     float* grid;                // [n_slots][nz][ny][nx]
+    const unsigned* n_live;     // optional (device): only slots < *n_live are live (device-driven fallback)
 };
 
 // ------------------------------------------------------------------ small helpers
@@ -241,19 +242,20 @@ struct VoxArgs {
     const int* atom_off;   // [n_probes + 1]
     const double* rot;     // [n_rot][9]
     const float* w;        // [P] weights folded into the grids
-    const int* unit_list;  // optional explicit units per slot (fallback); else unit_begin + slot
+    const int* unit_list;  // optional: slot -> call-relative unit (fallback); unit = unit_begin + unit_list[slot]
     long long unit_begin;
     int n_rot, n_slots, P, m;
     double spacing;
     float* Lw;             // [ceil(n_slots/RB)][P][m^3][RB]
     int* status;
+    const unsigned* n_live;   // optional (device): slots >= *n_live are zero padding (device-driven fallback)
 };
 
 // One thread per (slot, p): sums the coefficients of the probe's atoms in atom order
 // (deterministic), then multiplies by w_p.  Index math in FP64 with explicit IEEE
 // rounding (no FMA contraction) so that voxel indices equal the oracle's exactly.
 #ifndef DOCK_LAUNCHER_TU   // defined once, in dock.cu
-__global__ void k_voxelize(VoxArgs a)
+__device__ __forceinline__ void voxelize_body(const VoxArgs& a)
 {
     int idx = blockIdx.x * blockDim.x + threadIdx.x;
     const int n_pad = (a.n_slots + RB - 1) / RB * RB;   // the last batch is zero-padded
@@ -262,8 +264,9 @@ __global__ void k_voxelize(VoxArgs a)
     const int m = a.m, m3 = m * m * m;
     float* dst = a.Lw + (static_cast<size_t>(slot / RB) * a.P + p) * m3 * RB + (slot % RB);
     for (int v = 0; v < m3; v++) dst[v * RB] = 0.0f;
-    if (slot >= a.n_slots) return;
-    long long unit = a.unit_list ? static_cast<long long>(a.unit_list[slot]) : a.unit_begin + slot;
+    const int n_eff = a.n_live ? min(a.n_slots, static_cast<int>(*a.n_live)) : a.n_slots;
+    if (slot >= n_eff) return;
+    long long unit = a.unit_begin + (a.unit_list ? static_cast<long long>(a.unit_list[slot]) : slot);
     int probe = static_cast<int>(unit / a.n_rot), r = static_cast<int>(unit % a.n_rot);
     const double* q = a.rot + 9 * static_cast<size_t>(r);
 
@@ -308,6 +311,10 @@ __global__ void k_voxelize(VoxArgs a)
     const float wp = a.w[p];
     for (int v = 0; v < m3; v++) dst[v * RB] = dst[v * RB] * wp;
 }
+__global__ void k_voxelize(VoxArgs a) { voxelize_body(a); }
+// arguments read from device memory (the device-driven fallback's per-call arguments, so that a captured
+// CUDA graph of the fallback loop stays valid across calls)
+__global__ void k_voxelize_dyn(const VoxArgs* a) { voxelize_body(*a); }
 #endif
 
 // Lw [batch][P][m^3][RB]  ->  out [slot][P][m^3]   (debug export for dock_voxelize)
@@ -349,7 +356,9 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr(const __grid_constant__ CU
     const int tile_end = min(a.g.ntiles, tile_begin + a.tiles_per_region);
     const int n_it = (tile_end - tile_begin) * a.P;
     const int slot0 = batch * RB;
-    const int nb = min(RB, a.n_slots - slot0);
+    const int n_eff = a.n_live ? min(a.n_slots, static_cast<int>(*a.n_live)) : a.n_slots;
+    if (slot0 >= n_eff) return;   // uniform: a dead batch of the device-driven fallback
+    const int nb = min(RB, n_eff - slot0);
 
     uint64_t* full = reinterpret_cast<uint64_t*>(smem + a.nstage * a.stage_bytes);
     uint64_t* empty = full + a.nstage;
@@ -645,6 +654,24 @@ struct GreedyArgs {
     long long unit_begin;
     void* poses;
     unsigned flag_bits;         // pose flags of these picks: DOCK_POSE_FALLBACK (1) on the fallback path, 0 (FFT engine)
+    const unsigned* n_live;     // optional (device): grids >= *n_live are dead (device-driven fallback)
+    const struct FbDyn* dyn;    // optional (device): per-call poses / unit_begin / n_rot (device-driven fallback)
+};
+
+// Per-call arguments of the device-driven fallback, uploaded with the call's inputs (the captured fallback
+// graph reads them from device memory, so it stays valid across calls).
+struct FbDyn {
+    VoxArgs vox;                // voxelization of the flagged slots (unit_list = the chunk's slots)
+    void* poses;                // the call's dock_pose output
+    long long unit_begin;
+    int n_rot;
+    int pad_;
+};
+
+// Control block of the fallback loop: next flagged entry to process, live slots in this chunk.
+struct FbCtl {
+    unsigned pos;
+    unsigned n_live;
 };
 
 // One round j of the paper's best-then-exclude loop over full score grids,
@@ -656,6 +683,7 @@ __global__ void k_greedy_round(GreedyArgs a)
 {
     const int ctas_per_grid = gridDim.x / a.n;
     const int gi = blockIdx.x / ctas_per_grid, part = blockIdx.x % ctas_per_grid;
+    if (a.n_live && gi >= static_cast<int>(*a.n_live)) return;
     const float* S = a.grid + static_cast<size_t>(gi) * a.nx * a.ny * a.nz;
     const uint32_t ncell = static_cast<uint32_t>(a.nx) * a.ny * a.nz;
     unsigned long long* pk = a.picks + static_cast<size_t>(gi) * a.k;
@@ -697,13 +725,17 @@ __global__ void k_greedy_round(GreedyArgs a)
 __global__ void k_greedy_emit(GreedyArgs a)
 {
     const int i = blockIdx.x * blockDim.x + threadIdx.x;
-    if (i >= a.n * a.k) return;
+    const int n_eff = a.n_live ? min(a.n, static_cast<int>(*a.n_live)) : a.n;
+    if (i >= n_eff * a.k) return;
     const int gi = i / a.k, j = i % a.k;
+    void* poses = a.dyn ? a.dyn->poses : a.poses;
+    const long long unit_begin = a.dyn ? a.dyn->unit_begin : a.unit_begin;
+    const int n_rot = a.dyn ? a.dyn->n_rot : a.n_rot;
     const unsigned long long key = a.picks[static_cast<size_t>(gi) * a.k + j];
     const int slot = a.slots[gi];
-    const long long unit = a.unit_begin + slot;
+    const long long unit = unit_begin + slot;
     PoseOut po;
-    po.rot = static_cast<int32_t>(unit % a.n_rot);
+    po.rot = static_cast<int32_t>(unit % n_rot);
     if (key != KEY_MAX) {
         po.t_lin = static_cast<int32_t>(key & 0xffffffffu);
         po.score = unord_f32(static_cast<uint32_t>(key >> 32));
@@ -713,7 +745,35 @@ __global__ void k_greedy_emit(GreedyArgs a)
         po.score = __int_as_float(0x7fc00000);
         po.flags = a.flag_bits | 2u;
     }
-    reinterpret_cast<PoseOut*>(a.poses)[static_cast<size_t>(slot) * a.k + j] = po;
+    reinterpret_cast<PoseOut*>(poses)[static_cast<size_t>(slot) * a.k + j] = po;
+}
+#endif
+
+// ------------------------------------------------------------------ device-driven fallback loop
+//
+// The exact fallback runs as a CUDA graph: k_fb_init sets the loop condition from the
+// device-side flag count k_merge produced, and a conditional WHILE node repeats
+//   k_fb_chunk -> voxelize -> correlation (GRID epilogue) -> greedy rounds -> k_fb_advance
+// over chunks of `ch` flagged slots.  No host synchronisation is needed whatever the count.
+#ifndef DOCK_LAUNCHER_TU   // defined once, in dock.cu
+__global__ void k_fb_init(cudaGraphConditionalHandle h, const unsigned int* fb_cnt, FbCtl* ctl)
+{
+    ctl->pos = 0;
+    ctl->n_live = 0;
+    cudaGraphSetConditional(h, *fb_cnt > 0u ? 1u : 0u);
+}
+__global__ void k_fb_chunk(const unsigned int* fb_cnt, const int* fb_list, FbCtl* ctl, int* slots, int ch)
+{
+    const unsigned pos = ctl->pos, cnt = *fb_cnt;
+    const unsigned n = cnt > pos ? min(static_cast<unsigned>(ch), cnt - pos) : 0u;
+    for (int i = threadIdx.x; i < ch; i += blockDim.x) slots[i] = i < static_cast<int>(n) ? fb_list[pos + i] : 0;
+    if (threadIdx.x == 0) ctl->n_live = n;
+}
+__global__ void k_fb_advance(cudaGraphConditionalHandle h, const unsigned int* fb_cnt, FbCtl* ctl, int ch)
+{
+    const unsigned pos = ctl->pos + static_cast<unsigned>(ch);
+    ctl->pos = pos;
+    cudaGraphSetConditional(h, pos < *fb_cnt ? 1u : 0u);
 }
 #endif
 

@@ -69,6 +69,7 @@ struct TcArgs {
     unsigned long long* cand;
     // grid mode
     float* grid;
+    const unsigned* n_live;     // optional (device): rotations >= *n_live are dead (device-driven fallback)
     // diagnostics (DOCK_TC_TRACE / DOCK_TC_DEBUG environment variables; off on the product path):
     // trace = per-role cycle counters summed over CTAs (see TR_*); dbg 1 = epilogue skips the TMEM
     // drain, 2 = drain without candidate processing (timing experiments only: poses are invalid)
@@ -408,6 +409,8 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
 
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     const int block = blockIdx.x / a.G, region = blockIdx.x % a.G;
+    const int n_eff = a.n_live ? min(a.n_slots, static_cast<int>(*a.n_live)) : a.n_slots;
+    if (block * ROT >= n_eff) return;   // uniform: a dead block of the device-driven fallback
     const int tile_begin = region * a.tiles_per_region;
     const int tile_end = min(a.ntiles, tile_begin + a.tiles_per_region);
     const int n_tiles = tile_end - tile_begin;
@@ -641,7 +644,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
             const int nclass = a.nepi >> 2;
             const int r = quarter * 32 + lane;                  // rotation within the block (TMEM lane)
             const int slot = block * ROT + r;
-            const bool rot_ok = slot < a.n_slots;
+            const bool rot_ok = slot < n_eff;
             unsigned long long lst[LIST];
 #pragma unroll
             for (int i = 0; i < LIST; i++) lst[i] = KEY_MAX;
@@ -731,6 +734,8 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tcs(const __grid_constant_
 
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     const int block = blockIdx.x / a.G, region = blockIdx.x % a.G;
+    const int n_eff = a.n_live ? min(a.n_slots, static_cast<int>(*a.n_live)) : a.n_slots;
+    if (block * ROT >= n_eff) return;   // uniform: a dead block of the device-driven fallback
     const int tile_begin = region * a.tiles_per_region;
     const int tile_end = min(a.ntiles, tile_begin + a.tiles_per_region);
     const int n_tiles = tile_end - tile_begin;
@@ -904,7 +909,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tcs(const __grid_constant_
             const int nclass = a.nepi >> 2;
             const int r = quarter * 32 + lane;
             const int slot = block * ROT + r;
-            const bool rot_ok = slot < a.n_slots;
+            const bool rot_ok = slot < n_eff;
             unsigned long long lst[LIST];
 #pragma unroll
             for (int i = 0; i < LIST; i++) lst[i] = KEY_MAX;

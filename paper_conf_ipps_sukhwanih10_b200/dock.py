@@ -108,15 +108,28 @@ def dock_init(receptor, weights, spacing: float = 0.8, m_max: int = 8, device: i
     return DockContext(out.value, P, (nx, ny, nz), m_max, device, sh)
 
 
-def _probe_array(probes: Sequence[Any]):
+def _check_device(x, ctx: "DockContext", what: str):
+    """torch CUDA tensors must live on the context's device (the C side also rejects other devices)."""
+    if _is_torch(x) and x.is_cuda and x.device.index != ctx.device:
+        raise ValueError(f"{what} is on cuda:{x.device.index}, the context is on cuda:{ctx.device}")
+
+
+def _probe_array(probes: Sequence[Any], ctx: "DockContext"):
     keep: List[Any] = []
     arr = (N.dock_probe_desc * len(probes))()
     for i, p in enumerate(probes):
         xyz, coef, m = (p["xyz"], p["coef"], p["m"]) if isinstance(p, dict) else (p.xyz, p.coef, p.m)
+        _check_device(xyz, ctx, f"probe {i} xyz")
+        _check_device(coef, ctx, f"probe {i} coef")
         xp, xk = _buf(xyz, "f8")
         cp, ck = _buf(coef, "f4")
         keep += [xk, ck]
         n_atoms = int(xk.shape[0]) if xk.ndim >= 1 else 0
+        # the C side reads n_atoms x 3 doubles and n_atoms x P floats: reject anything else here
+        if tuple(xk.shape) != (n_atoms, 3):
+            raise ValueError(f"probe {i}: xyz must be [n_atoms][3], got {tuple(xk.shape)}")
+        if tuple(ck.shape) not in ((n_atoms, ctx.P),) and not (n_atoms == 0 and ck.size == 0):
+            raise ValueError(f"probe {i}: coef must be [n_atoms][P] = [{n_atoms}][{ctx.P}], got {tuple(ck.shape)}")
         arr[i] = N.dock_probe_desc(n_atoms, int(m), C.c_void_p(xp if n_atoms else None),
                                    C.c_void_p(cp if n_atoms else None))
     return arr, keep
@@ -129,6 +142,8 @@ def _alloc_poses(n_units: int, k: int, out, device: int):
     if _is_torch(out):
         if out.dtype != _torch().int32 or tuple(out.shape) != (n_units, k, 4) or not out.is_contiguous():
             raise ValueError("device pose buffer must be a contiguous int32 tensor [U][k][4]")
+        if out.is_cuda and out.device.index != device:
+            raise ValueError(f"pose buffer is on cuda:{out.device.index}, the context is on cuda:{device}")
         return out, out.data_ptr()
     if out.dtype != POSE_DTYPE or out.shape != (n_units, k) or not out.flags.c_contiguous:
         raise ValueError("host pose buffer must be a contiguous POSE_DTYPE array [U][k]")
@@ -139,15 +154,18 @@ def dock_probe_batch(ctx: DockContext, probes: Sequence[Any], rot, unit_begin: i
                      unit_end: Optional[int] = None, k: int = 4, rho: int = 1, out=None):
     """Dock probe-major (probe, rotation) units [unit_begin, unit_end); the hot path.
 
-    ``out``: None -> a host numpy POSE_DTYPE array [U][k]; or a caller buffer (numpy POSE_DTYPE
-    [U][k], or an int32 torch tensor [U][k][4] on the context's device -> device-resident output).
+    ``out``: None -> a host numpy POSE_DTYPE array [U][k] (synchronous); or a caller buffer (numpy
+    POSE_DTYPE [U][k], synchronous; or an int32 torch tensor [U][k][4] on the context's device ->
+    device-resident output, ASYNCHRONOUS: the call returns once the work is enqueued on the context's
+    stream; call ``dock_sync`` for device-detected errors, see include/dock.h).
     """
     torch = _torch()
     n_rot = int(rot.shape[0])
     if unit_end is None:
         unit_end = len(probes) * n_rot
+    _check_device(rot, ctx, "rot")
     rp, rk = _buf(rot, "f8")
-    arr, keep = _probe_array(probes)
+    arr, keep = _probe_array(probes, ctx)
     o, op = _alloc_poses(unit_end - unit_begin, k, out, ctx.device)
     with torch.cuda.device(ctx.device):
         st = N.lib().dock_probe_batch(ctx.ptr, arr, len(probes), C.c_void_p(rp), n_rot, int(unit_begin),
@@ -155,6 +173,15 @@ def dock_probe_batch(ctx: DockContext, probes: Sequence[Any], rot, unit_begin: i
     _check(ctx.ptr, st)
     del rk, keep
     return o
+
+
+def dock_sync(ctx: DockContext):
+    """Sync point of the asynchronous (device-output) calls: waits for the context's stream and raises
+    DockError for a device-detected error of any call since the previous sync point."""
+    torch = _torch()
+    with torch.cuda.device(ctx.device):
+        st = N.lib().dock_sync(ctx.ptr)
+    _check(ctx.ptr, st)
 
 
 def dock_probe(ctx: DockContext, probe, rot, k: int = 4, rho: int = 1, out=None):
@@ -169,7 +196,7 @@ def dock_score_grid(ctx: DockContext, probe, rot9, per_term: bool = False):
     S = np.zeros((nz, ny, nx), np.float32)
     C_ = np.zeros((ctx.P, nz, ny, nx), np.float32) if per_term else None
     rp, rk = _buf(np.asarray(rot9, dtype=np.float64).reshape(9) if not _is_torch(rot9) else rot9, "f8")
-    arr, keep = _probe_array([probe])
+    arr, keep = _probe_array([probe], ctx)
     with torch.cuda.device(ctx.device):
         st = N.lib().dock_score_grid(ctx.ptr, arr, C.c_void_p(rp), C.c_void_p(S.ctypes.data),
                                      C.c_void_p(C_.ctypes.data if per_term else None))
@@ -184,7 +211,7 @@ def dock_voxelize(ctx: DockContext, probe, rot):
     n_rot = int(rot.shape[0])
     out = np.zeros((n_rot, ctx.P, m, m, m), np.float32)
     rp, rk = _buf(rot, "f8")
-    arr, keep = _probe_array([probe])
+    arr, keep = _probe_array([probe], ctx)
     with torch.cuda.device(ctx.device):
         st = N.lib().dock_voxelize(ctx.ptr, arr, C.c_void_p(rp), n_rot, C.c_void_p(out.ctypes.data))
     _check(ctx.ptr, st)

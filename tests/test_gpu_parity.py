@@ -362,9 +362,100 @@ def test_device_resident_io(D):
                for p in probes]
     out = torch.empty((len(probes) * len(rot), 4, 4), dtype=torch.int32, device="cuda")
     D.dock_probe_batch(ctx, dprobes, torch.from_numpy(rot).cuda(), k=4, rho=1, out=out)
-    torch.cuda.synchronize()
+    D.dock_sync(ctx)
     assert np.array_equal(D.poses_from_device(out), host)
     ctx.close()
+
+
+@pytest.mark.parametrize("engine", ENGINES)
+def test_async_device_output_and_fallback_loop(D, engine):
+    """Device output is asynchronous: many calls are queued back to back without a host sync (the exact
+    fallback runs as a device-driven CUDA-graph loop over chunks of flagged rotations).  Forcing every
+    rotation of 150 units through that loop (several chunks: 128 per chunk on the tensor cores, 64 on
+    FFMA) returns the same pose bits as the candidate path, and queued calls equal one-at-a-time calls."""
+    import torch
+    P, m = 4, 4
+    R = g.receptor_ftmap_like((48, 40, 36), P)
+    w = g.weights(P)
+    probes = g.probes(3, m, P)
+    rot = g.rotations(50)
+    n = len(probes) * len(rot)
+    ctx = _ctx(D, R, w, m, engine)
+    ref = D.dock_probe_batch(ctx, probes, rot, k=4, rho=1)
+    assert _engine_id(D.dock_get_info(ctx)) == engine
+    dprobes = [{"xyz": torch.from_numpy(p.xyz).cuda(), "coef": torch.from_numpy(p.coef).cuda(), "m": p.m}
+               for p in probes]
+    drot = torch.from_numpy(rot).cuda()
+    outs = [torch.full((n, 4, 4), -7, dtype=torch.int32, device="cuda") for _ in range(3)]
+    D.dock_set_tuning(ctx, D.DOCK_TUNE_FORCE_FALLBACK, 1)
+    D.dock_probe_batch(ctx, dprobes, drot, k=4, rho=1, out=outs[0])   # returns before the GPU finishes
+    D.dock_set_tuning(ctx, D.DOCK_TUNE_FORCE_FALLBACK, 0)
+    D.dock_probe_batch(ctx, dprobes, drot, k=4, rho=1, out=outs[1])
+    D.dock_probe_batch(ctx, probes, rot, 10, n, k=4, rho=1, out=outs[2][10:])   # host inputs, async output
+    D.dock_sync(ctx)
+    forced, plain, part = (D.poses_from_device(o) for o in outs)
+    assert (forced["flags"] & D.DOCK_POSE_FALLBACK).all()
+    for got in (forced, plain):
+        assert np.array_equal(got["t_lin"], ref["t_lin"])
+        assert np.array_equal(got["score"].view(np.uint32), ref["score"].view(np.uint32))
+    assert np.array_equal(part[10:]["t_lin"], ref[10:]["t_lin"])
+    assert (outs[2][:10] == -7).all()
+    info = D.dock_get_info(ctx)
+    assert info["pending"] == 0
+    ctx.close()
+
+
+def test_async_errors_surface_at_sync(D):
+    """A device-detected input error of an asynchronous call is reported by dock_sync (and is cleared)."""
+    import torch
+    P = 1
+    R = g.receptor_uniform((16, 16, 16), P)
+    ctx = D.dock_init(R, np.ones(P, np.float32), H, m_max=4)
+    pr = g.probe(0, 4, P)
+    out = torch.empty((1, 1, 4), dtype=torch.int32, device="cuda")
+    D.dock_probe_batch(ctx, [pr], np.diag([1.0, 1.0, -1.0]).reshape(1, 9), k=1, rho=0, out=out)   # no raise
+    with pytest.raises(D.DockError) as e:
+        D.dock_sync(ctx)
+    assert e.value.status == -4
+    D.dock_sync(ctx)   # cleared
+    far = g.Probe(np.array([[4.0, 0, 0]]), np.ones((1, 1), np.float32), 4)
+    out3 = torch.empty((3, 1, 4), dtype=torch.int32, device="cuda")
+    D.dock_probe_batch(ctx, [far], g.rotations(3), k=1, rho=0, out=out3)
+    D.dock_probe_batch(ctx, [pr], g.rotations(3), k=1, rho=0, out=out3)   # a later good call does not hide it
+    with pytest.raises(D.DockError) as e:
+        D.dock_sync(ctx)
+    assert e.value.status == -3
+    ctx.close()
+
+
+def test_sharded_one_rank_nccl(D):
+    """The multi-GPU data plane under a 1-rank NCCL group: the docking call writes into this rank's slot of
+    the preallocated all-gather buffer and one in-place NCCL all-gather returns the poses, bitwise equal to
+    dock_probe_batch."""
+    import os
+    import socket
+    import torch
+    import torch.distributed as dist
+    from paper_conf_ipps_sukhwanih10_b200 import parallel
+    sock = socket.socket()
+    sock.bind(("127.0.0.1", 0))
+    port = sock.getsockname()[1]
+    sock.close()
+    os.environ.update(MASTER_ADDR="127.0.0.1", MASTER_PORT=str(port))
+    dist.init_process_group("nccl", rank=0, world_size=1, device_id=torch.device("cuda", 0))
+    try:
+        P, m = 4, 4
+        R = g.receptor_ftmap_like((40, 32, 32), P)
+        probes = g.probes(2, m, P)
+        rot = g.rotations(11)
+        ctx = D.dock_init(R, g.weights(P), H, m_max=m, device=0)
+        ref = D.dock_probe_batch(ctx, probes, rot, k=4, rho=1)
+        for _ in range(2):   # the second call reuses the cached buffer
+            full = parallel.dock_probe_sharded(ctx, probes, rot, k=4, rho=1)
+            assert np.array_equal(D.poses_from_device(full), ref)
+        ctx.close()
+    finally:
+        dist.destroy_process_group()
 
 
 def test_errors(D):
