@@ -70,6 +70,13 @@ typedef enum {
 #define DOCK_MAX_M 8       /* probe grid edge m <= 8 (paper: <= 8^3 in constant memory) */
 #define DOCK_MAX_K 32      /* poses kept per rotation (FTMap: 4) */
 
+/* Engines (DOCK_TUNE_ENGINE) */
+#define DOCK_ENGINE_AUTO 0
+#define DOCK_ENGINE_FFMA 1
+#define DOCK_ENGINE_TC 2
+#define DOCK_ENGINE_FFT 3
+#define DOCK_ENGINE_SPARSE 4
+
 /* Pose flags */
 #define DOCK_POSE_FALLBACK 1u   /* exact full-grid fallback was used for this rotation */
 #define DOCK_POSE_EMPTY 2u      /* fewer than k translations were available (never with valid args) */
@@ -92,7 +99,9 @@ typedef struct {
     int device;       /* CUDA device ordinal */
     double spacing;   /* grid spacing h in Angstrom (> 0, finite); BASELINE uses 0.8.  double so that the
                          kernel divides by exactly the caller's h, as the FP64 oracle does (reading Q18) */
-    void* stream;     /* cudaStream_t to run on; NULL => the context creates its own */
+    void* stream;     /* cudaStream_t to run on (cudaStreamLegacy / cudaStreamPerThread allowed); NULL => the
+                         context creates its own non-blocking stream (work of other streams is then NOT ordered
+                         with the context's: the caller synchronises) */
 } dock_grid_desc;
 
 /* One probe (small molecule). */
@@ -155,7 +164,11 @@ typedef enum {
     DOCK_TUNE_ENGINE = 4,         /* correlation engine: 0 auto (tcgen05 when eligible), 1 FP32 FFMA, 2 tcgen05,
                                      3 FFT (cuFFT R2C/C2R + this library's channel multiply-accumulate and exact
                                      greedy on the score grids; the paper's FFT method P:L156-163, kept as the
-                                     comparison point of the direct-vs-FFT crossover P:L485-502; never auto) */
+                                     comparison point of the direct-vs-FFT crossover P:L485-502; never auto),
+                                     4 sparse ligand (FP32 direct correlation over the occupied probe voxels only:
+                                     per-probe atom grids G_a = sum_p w_p coef_ap R_p gathered at each atom's voxel,
+                                     P:L504-509, L553-555; needs <= 32 atoms per probe; auto picks it by a cost
+                                     model) */
     DOCK_TUNE_TC_VARIANT = 5,     /* tcgen05 kernel: 0 auto, 1 = resident receptor boxes (one channel group, P <= 4,
                                      128 translations x 4 rows per tile), 2 = receptor streamed one (channel group,
                                      z-plane) unit at a time (any P <= 32, m <= 8; 64 / 128 / 160 translations per
@@ -180,7 +193,7 @@ typedef struct {
     double l2_bytes;           /* device L2 size (cudaDevAttrL2CacheSize) */
     double corr_ms_last;       /* CUDA-event duration of the last k_corr launch (dock_probe_batch), -1 if none */
     int n_sms;                 /* multiprocessors of the context's device */
-    int engine_last;           /* engine of the last correlation: 1 FP32 FFMA, 2 tcgen05 bf16x3, 3 FFT */
+    int engine_last;           /* engine of the last correlation: 1 FP32 FFMA, 2 tcgen05 bf16x3, 3 FFT, 4 sparse */
     int tc_available;          /* 1 if the tcgen05 engine is available for m_max */
     int tc_variant_last;       /* tcgen05 variant of the last correlation (1 or 2), 0 if FFMA */
     int tc_ksteps_last;        /* K-steps (K = 16 each) per translation row executed by the last tcgen05 launch */
@@ -188,6 +201,9 @@ typedef struct {
     int tc_rows_per_tile_last; /* translation rows per tile (TMEM accumulators) of the last tcgen05 launch */
     int pending;               /* 1 if the last asynchronous call has not reached a sync point (dock_sync) */
     int fb_chunk;              /* flagged rotations per iteration of the device-driven fallback loop */
+    int sp_atom_grids_last;    /* sparse engine: atom grids G_a computed by the last call */
+    int sp_row_last;           /* sparse engine: translations per column row (32 x per-lane count) */
+    double sp_terms_last;      /* sparse engine: atoms summed over the units of the last call (gathers per translation) */
 } dock_info;
 
 dock_status dock_get_info(const dock_ctx* ctx, dock_info* info);

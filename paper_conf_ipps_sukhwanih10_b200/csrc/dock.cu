@@ -20,6 +20,7 @@
 #include "dock.h"
 #include "dock_kernels.cuh"
 #include "dock_tc.cuh"
+#include "dock_sparse.cuh"
 #include "dock_launch.h"
 #include "dock_fft.h"
 
@@ -43,6 +44,14 @@ struct TcPlan {                // per-(variant, probe size) plan of the tcgen05 
     int box_bytes = 0, box_bytes_pair = 0, rec_stage_bytes = 0, n_rec_stages = 0, smem = 0, nsteps = 0, wstages = 0;
     int TXBP = 0;              // variant 1: x extent of the pair box (the main box uses TXB of make_tc_plan)
 };
+
+struct SpPlan {                // per-probe-size plan of the sparse-ligand engine (dock_sparse.cuh)
+    bool ok = false;
+    int xts = 0, TX = 0, ntx = 0, nty = 0, TXB = 0, TYB = 0, slot_words = 0, box_bytes = 0;
+    int GXp = 0, GYp = 0, GZp = 0;   // padded atom-grid extents (cyclic halo materialised)
+};
+
+enum EngineKind { ENG_FFMA = 1, ENG_TC = 2, ENG_FFT = 3, ENG_SPARSE = 4 };
 
 struct MPlan {                 // per-probe-size launch plan
     bool ok = false;
@@ -107,8 +116,15 @@ struct dock_ctx {
     // device-driven exact fallback (a CUDA graph with a WHILE node over chunks of flagged slots)
     cudaStream_t cap_stream = nullptr, cap_stream2 = nullptr;   // private capture streams
     cudaGraphExec_t fb_exec = nullptr;
-    unsigned char fb_key[128] = {0};
-    DevBuf fb_grid, fb_Lw, fb_W, fb_picks, fb_slots, fb_ctl;
+    unsigned char fb_key[256] = {0};
+    DevBuf fb_grid, fb_Lw, fb_W, fb_picks, fb_slots, fb_ctl, fb_groups;
+    // sparse-ligand engine: plans, atom grids G_a of the call, occupied-voxel term tables
+    SpPlan spplan[DOCK_MAX_M + 1][6];   // [m][xts]
+    DevBuf sp_G, sp_tv, sp_ts, sp_nt, sp_dw, sp_slot_atoms;
+    CUtensorMap sp_tmap;
+    int sp_natoms_last = 0;           // atom grids of the last sparse call
+    int sp_tx_last = 0;
+    double sp_terms_last = 0;         // occupied voxels summed over the units of the last sparse call
     // tuning
     int regions_override = 0;
     int force_fallback = 0;
@@ -449,7 +465,8 @@ dock_status check_ctx(dock_ctx* ctx)
 // *d_fb receives their device address.
 dock_status stage_inputs(dock_ctx* ctx, const dock_probe_desc* probes, int n_probes, const double* rot,
                          int n_rot, const double** d_xyz, const float** d_coef, const int** d_off,
-                         const double** d_rot, dk::FbDyn* fb = nullptr, const dk::FbDyn** d_fb = nullptr)
+                         const double** d_rot, dk::FbDyn* fb = nullptr, const dk::FbDyn** d_fb = nullptr,
+                         const void* extra = nullptr, size_t extra_bytes = 0, const void** d_extra = nullptr)
 {
     // One pinned staging block [fb args][off][gather table][rot (host)][host xyz][host coef] goes up in a
     // single H2D copy; one gather kernel then assembles all probes' atoms (device-resident probe arrays are
@@ -466,7 +483,8 @@ dock_status stage_inputs(dock_ctx* ctx, const dock_probe_desc* probes, int n_pro
     const size_t b_xyz = sizeof(double) * 3 * std::max(na, 1), b_coef = sizeof(float) * P * std::max(na, 1);
     const size_t o_off = b_fb, o_tab = o_off + (b_off + 15) / 16 * 16, o_rot = o_tab + (b_tab + 15) / 16 * 16;
     const size_t o_xyz = o_rot + (b_rot + 15) / 16 * 16, o_coef = o_xyz + (b_xyz + 15) / 16 * 16;
-    const size_t total = o_coef + b_coef;
+    const size_t o_extra = o_coef + (b_coef + 15) / 16 * 16;   // optional blob (sparse engine: group table)
+    const size_t total = o_extra + extra_bytes;
     TRY(ensure(ctx, ctx->xyz, b_xyz));
     TRY(ensure(ctx, ctx->coef, b_coef));
     TRY(ensure(ctx, ctx->off, total));   // device copy of the whole staging block
@@ -506,6 +524,10 @@ dock_status stage_inputs(dock_ctx* ctx, const dock_probe_desc* probes, int n_pro
     *d_xyz = static_cast<const double*>(ctx->xyz.p);
     *d_coef = static_cast<const float*>(ctx->coef.p);
     *d_off = reinterpret_cast<const int*>(ds + o_off);
+    if (extra_bytes) {
+        memcpy(hs + o_extra, extra, extra_bytes);
+        *d_extra = ds + o_extra;
+    }
     if (fb) {
         fb->vox.xyz = *d_xyz;
         fb->vox.coef = *d_coef;
@@ -659,16 +681,255 @@ bool plan_tc_launch(dock_ctx* ctx, int m, int n_slots, int* v_out, int* G_out)
     return true;
 }
 
-// Engine choice: tensor cores when a plan for this m exists (auto) or when forced.
-dock_status select_engine(dock_ctx* ctx, int m, bool* use_tc)
+// Engine choice.  Forced: 1 FFMA, 2 tcgen05, 4 sparse ligand (DOCK_E_UNSUPPORTED when ineligible).  Auto:
+// the sparse-ligand engine when it is eligible and its cost model (one gathered value per occupied voxel and
+// translation) beats the dense engine's, else tcgen05 when a plan exists for m, else FFMA.
+dock_status select_engine(dock_ctx* ctx, int m, bool sparse_ok, bool sparse_better, int* kind)
 {
     int v = 0, G = 0;
-    const bool ok = plan_tc_launch(ctx, m, tc::ROT, &v, &G);
-    if (ctx->engine == 2 && !ok) return fail(ctx, DOCK_E_UNSUPPORTED, "tensor-core engine unavailable for m=%d", m);
-    *use_tc = ctx->engine == 2 || (ctx->engine == 0 && ok);
-    ctx->engine_last = *use_tc ? 2 : 1;
-    if (!*use_tc) ctx->tc_variant_last = 0;
+    const bool tc_ok = plan_tc_launch(ctx, m, tc::ROT, &v, &G);
+    if (ctx->engine == 2 && !tc_ok) return fail(ctx, DOCK_E_UNSUPPORTED, "tensor-core engine unavailable for m=%d", m);
+    if (ctx->engine == 4 && !sparse_ok)
+        return fail(ctx, DOCK_E_UNSUPPORTED, "sparse-ligand engine ineligible (atoms per probe or shared memory)");
+    int k = ENG_FFMA;
+    if (ctx->engine == 1) k = ENG_FFMA;
+    else if (ctx->engine == 2) k = ENG_TC;
+    else if (ctx->engine == 4) k = ENG_SPARSE;
+    else k = (sparse_ok && sparse_better) ? ENG_SPARSE : tc_ok ? ENG_TC : ENG_FFMA;
+    *kind = k;
+    ctx->engine_last = k;
+    if (k != ENG_TC) ctx->tc_variant_last = 0;
     return DOCK_OK;
+}
+
+// ---------------------------------------------------------------- sparse-ligand engine (dock_sparse.cuh)
+
+dock_status make_sp_plan(dock_ctx* ctx, int m, int xts)
+{
+    SpPlan& pl = ctx->spplan[m][xts];
+    if (pl.ok) return DOCK_OK;
+    pl.xts = xts;
+    pl.TX = 32 * pl.xts;
+    pl.TXB = round_up(pl.TX + m - 1, 4);
+    pl.TYB = sp::TY + m - 1;
+    if (pl.TXB > 256 || pl.TYB > 256) return fail(ctx, DOCK_E_UNSUPPORTED, "sparse engine: TMA box too large");
+    pl.ntx = (ctx->nx + pl.TX - 1) / pl.TX;
+    pl.nty = (ctx->ny + sp::TY - 1) / sp::TY;
+    pl.slot_words = round_up(pl.TXB * pl.TYB, 32);
+    pl.box_bytes = pl.TXB * pl.TYB * 4;
+    pl.GXp = round_up((pl.ntx - 1) * pl.TX + pl.TXB, 4);
+    pl.GYp = (pl.nty - 1) * sp::TY + pl.TYB;
+    pl.GZp = ctx->nz + m - 1;
+    pl.ok = true;
+    return DOCK_OK;
+}
+
+// Plane-ring depth for tmax atoms: as deep as shared memory allows (<= NPLMAX planes: the steps beyond the
+// window m + PZ - 1 are TMA prefetch), at least the window; 0 when not even that fits.
+int sp_npl(const SpPlan& pl, int m, int tmax)
+{
+    const int budget = kSmemLimit - 22 * 1024;   // static shared memory of k_corr_sparse: ~20 KB (lists, terms)
+    for (int npl = sp::NPLMAX; npl >= m + sp::PZ - 1; npl--)
+        if ((size_t)std::max(tmax, 1) * npl * pl.slot_words * 4 <= (size_t)budget) return npl;
+    return 0;
+}
+
+struct SpCall {   // one sparse-engine launch over the units of a call
+    bool ok = false;
+    int xts = 0;                      // translations per lane along x (row width 32 * xts)
+    int m = 0, tmax = 0, n_at = 0, atom_lo = 0, npl = 0, smem = 0;
+    double terms = 0;                 // estimated occupied voxels summed over the units (cost model)
+    std::vector<sp::Group> groups;    // rotation groups (<= sp::RB rotations of one probe)
+};
+
+// Host-side plan of a sparse-engine call: atom range of the probes the units touch, rotation groups,
+// eligibility (atoms per probe <= sp::TMAX, plane ring fits shared memory).
+dock_status sp_prepare(dock_ctx* ctx, int m, const dock_probe_desc* probes, int n_probes, int n_rot,
+                       int64_t unit_begin, int64_t unit_end, SpCall* sc)
+{
+    sc->ok = false;
+    sc->groups.clear();
+    if (unit_end <= unit_begin) return DOCK_OK;
+    const int p_lo = (int)(unit_begin / n_rot), p_hi = (int)((unit_end - 1) / n_rot);
+    int atoms = 0, tmax = 0;
+    std::vector<int> base(p_hi - p_lo + 1);
+    for (int p = p_lo; p <= p_hi; p++) {
+        base[p - p_lo] = atoms;
+        atoms += probes[p].n_atoms;
+        tmax = std::max(tmax, probes[p].n_atoms);
+    }
+    if (tmax > sp::TMAX) return DOCK_OK;
+    // row width: the fewest wasted x translations whose plane ring fits shared memory for tmax atoms
+    // (ties: 128, then 160, then 64 translations per row)
+    int xts = 0, npl = 0, best_w = 1 << 30;
+    for (int x : {4, 5, 2}) {
+        if (make_sp_plan(ctx, m, x) != DOCK_OK) continue;
+        const int n = sp_npl(ctx->spplan[m][x], m, tmax);
+        const int w = (ctx->nx + 32 * x - 1) / (32 * x) * (32 * x);
+        if (n && w < best_w) {
+            best_w = w;
+            xts = x;
+            npl = n;
+        }
+    }
+    cudaGetLastError();
+    ctx->err[0] = 0;
+    if (!xts) return DOCK_OK;   // ineligible, not an error
+    const SpPlan& pl = ctx->spplan[m][xts];
+    sc->xts = xts;
+    int off = 0;
+    for (int p = 0; p < p_lo; p++) off += probes[p].n_atoms;
+    sc->m = m;
+    sc->tmax = tmax;
+    sc->n_at = atoms;
+    sc->atom_lo = off;
+    sc->npl = npl;
+    sc->smem = std::max(tmax, 1) * npl * pl.slot_words * 4;
+    sc->terms = 0;
+    for (int p = p_lo; p <= p_hi; p++) {
+        const int64_t u0 = std::max<int64_t>(unit_begin, (int64_t)p * n_rot);
+        const int64_t u1 = std::min<int64_t>(unit_end, (int64_t)(p + 1) * n_rot);
+        sc->terms += double(u1 - u0) * probes[p].n_atoms;
+        for (int64_t u = u0; u < u1; u += sp::RB) {
+            sp::Group gr;
+            gr.slot0 = (int)(u - unit_begin);
+            gr.n = (int)std::min<int64_t>(sp::RB, u1 - u);
+            gr.atom0 = base[p - p_lo];
+            gr.n_atoms = probes[p].n_atoms;
+            sc->groups.push_back(gr);
+        }
+    }
+    sc->ok = true;
+    return DOCK_OK;
+}
+
+// Cost model of the engine choice (auto): gathered values per SM-clock of the sparse engine vs executed
+// bf16 MACs per SM-clock of the tensor-core engine (bf16x3 with the PAIR scheme: 3 per algorithmic MAC),
+// both measured on B200: ~6 gathers and ~3000 MACs per clock and SM.
+bool sp_better(const dock_ctx* ctx, const SpCall& sc, int m, int n_units)
+{
+    if (!sc.ok) return false;
+    const double ncell = (double)ctx->nx * ctx->ny * ctx->nz;
+    const double sparse = sc.terms * ncell / 6.0;
+    const double dense = double(n_units) * ncell * ctx->P * m * m * m * 3.0 / 3000.0;
+    return sparse < dense;
+}
+
+// Columns per item: minimise waves * (columns per item + per-item overhead, ~1 column: list warm-up and
+// pipeline fill)
+int sp_choose_cols(const dock_ctx* ctx, const SpPlan& pl, int64_t n_groups)
+{
+    const int ncol = pl.ntx * pl.nty;
+    if (ctx->regions_override > 0) {   // DOCK_TUNE_REGIONS: regions (items) per rotation group
+        const int G = std::min(ctx->regions_override, ncol);
+        return (ncol + G - 1) / G;
+    }
+    int best = ncol;
+    double best_cost = 1e300;
+    for (int G = 1; G <= ncol; G++) {
+        const int cpi = (ncol + G - 1) / G;
+        const int geff = (ncol + cpi - 1) / cpi;
+        const int64_t items = n_groups * geff;
+        const int64_t waves = (items + ctx->n_sms - 1) / ctx->n_sms;
+        const double cost = double(waves) * (cpi + 1.0);
+        if (cost < best_cost - 1e-9) {
+            best_cost = cost;
+            best = cpi;
+        }
+    }
+    return best;
+}
+
+// Per call: atom grids G_a of the touched probes (weights w) + their tensor map, and the occupied-voxel
+// term tables of every unit.
+dock_status sp_run_pre(dock_ctx* ctx, const SpCall& sc, int n_slots, int64_t unit_begin, int n_rot,
+                       const double* d_xyz, const float* d_coef, const int* d_off, const double* d_rot, const float* w)
+{
+    const SpPlan& pl = ctx->spplan[sc.m][sc.xts];
+    const size_t gcells = (size_t)pl.GXp * pl.GYp * pl.GZp;
+    TRY(ensure(ctx, ctx->sp_G, sizeof(float) * gcells * std::max(sc.n_at, 1)));
+    TRY(ensure(ctx, ctx->sp_tv, sizeof(int) * (size_t)n_slots * sp::TMAX));
+    TRY(ensure(ctx, ctx->sp_ts, sizeof(int) * (size_t)n_slots * sp::TMAX));
+    TRY(ensure(ctx, ctx->sp_nt, sizeof(int) * (size_t)n_slots));
+    TRY(ensure(ctx, ctx->sp_dw, sizeof(float) * (size_t)n_slots * sp::TMAX * ctx->P));
+    TRY(ensure(ctx, ctx->sp_slot_atoms, sizeof(int) * 2 * (size_t)n_slots));
+    auto fn = encode_fn();
+    if (!fn) return fail(ctx, DOCK_E_CUDA, "cuTensorMapEncodeTiled unavailable");
+    cuuint64_t dims[4] = {(cuuint64_t)pl.GXp, (cuuint64_t)pl.GYp, (cuuint64_t)pl.GZp,
+                          (cuuint64_t)std::max(sc.n_at, 1)};
+    cuuint64_t strides[3] = {(cuuint64_t)pl.GXp * 4, (cuuint64_t)pl.GXp * pl.GYp * 4, (cuuint64_t)gcells * 4};
+    cuuint32_t box[4] = {(cuuint32_t)pl.TXB, (cuuint32_t)pl.TYB, 1, 1};
+    cuuint32_t es[4] = {1, 1, 1, 1};
+    CUresult r = fn(&ctx->sp_tmap, CU_TENSOR_MAP_DATA_TYPE_FLOAT32, 4, ctx->sp_G.p, dims, strides, box, es,
+                    CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_L2_256B,
+                    CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+    if (r != CUDA_SUCCESS) return fail(ctx, DOCK_E_CUDA, "cuTensorMapEncodeTiled (atom grids) failed (%d)", (int)r);
+    if (sc.n_at > 0) {
+        const size_t n4 = gcells / 4 * sc.n_at;
+        const int blocks = (int)std::min<size_t>((n4 + 255) / 256, (size_t)ctx->n_sms * 16);
+        sp::k_atom_grids<<<blocks, 256, 0, ctx->stream>>>(ctx->d_rec, ctx->geo.Xp, ctx->geo.Yp, ctx->geo.Zp, ctx->nx,
+                                                         ctx->ny, ctx->nz, ctx->P, d_coef, w, sc.atom_lo, sc.n_at,
+                                                         static_cast<float*>(ctx->sp_G.p), pl.GXp, pl.GYp, pl.GZp);
+        CU(cudaGetLastError());
+        ctx->kernels_last++;
+    }
+    sp::SpVoxArgs v{};
+    v.xyz = d_xyz;
+    v.coef = d_coef;
+    v.atom_off = d_off;
+    v.rot = d_rot;
+    v.w = w;
+    v.unit_begin = unit_begin;
+    v.n_rot = n_rot;
+    v.n_slots = n_slots;
+    v.P = ctx->P;
+    v.m = sc.m;
+    v.spacing = ctx->spacing;
+    v.term_v = static_cast<int*>(ctx->sp_tv.p);
+    v.term_src = static_cast<int*>(ctx->sp_ts.p);
+    v.n_terms = static_cast<int*>(ctx->sp_nt.p);
+    v.dw = static_cast<float*>(ctx->sp_dw.p);
+    v.status = ctx->d_small;
+    v.slot_atoms = static_cast<int*>(ctx->sp_slot_atoms.p);
+    v.atom_lo = sc.atom_lo;
+    sp::k_voxelize_sparse<<<(n_slots + 127) / 128, 128, 0, ctx->stream>>>(v);
+    CU(cudaGetLastError());
+    ctx->kernels_last++;
+    ctx->sp_natoms_last = sc.n_at;
+    ctx->sp_tx_last = pl.TX;
+    ctx->sp_terms_last = sc.terms;
+    return DOCK_OK;
+}
+
+sp::SpArgs sp_args(dock_ctx* ctx, const SpCall& sc, const sp::Group* d_groups, int64_t n_groups)
+{
+    const SpPlan& pl = ctx->spplan[sc.m][sc.xts];
+    sp::SpArgs a{};
+    a.nx = ctx->nx;
+    a.ny = ctx->ny;
+    a.nz = ctx->nz;
+    a.m = sc.m;
+    a.TX = pl.TX;
+    a.ntx = pl.ntx;
+    a.nty = pl.nty;
+    a.TXB = pl.TXB;
+    a.TYB = pl.TYB;
+    a.slot_words = pl.slot_words;
+    a.npl = sc.npl;
+    a.cols_per_item = sp_choose_cols(ctx, pl, n_groups);
+    a.G = (pl.ntx * pl.nty + a.cols_per_item - 1) / a.cols_per_item;
+    a.box_bytes = pl.box_bytes;
+    a.groups = d_groups;
+    a.term_v = static_cast<const int*>(ctx->sp_tv.p);
+    a.term_src = static_cast<const int*>(ctx->sp_ts.p);
+    a.n_terms = static_cast<const int*>(ctx->sp_nt.p);
+    a.dw = static_cast<const float*>(ctx->sp_dw.p);
+    a.P = ctx->P;
+    a.rec = ctx->d_rec;
+    a.rXp = ctx->geo.Xp;
+    a.rYp = ctx->geo.Yp;
+    a.rZp = ctx->geo.Zp;
+    return a;
 }
 
 // Pack folded FP32 weights into the tcgen05 A-operand layout of variant v.
@@ -777,13 +1038,16 @@ dock_status run_grid_tc(dock_ctx* ctx, int m, int n_slots, const float* Lw, floa
 // across calls with the same shape; the host never waits for the flag count.
 
 struct FbKey {   // everything the captured fallback graph bakes in (compared bytewise)
-    int m, use_tc, v, G, k, rho, ch, nepi, P, nx, ny, nz;
+    int m, kind, v, G, k, rho, ch, nepi, P, nx, ny, nz;
+    int sp_nat, sp_npl, sp_smem, sp_xts;
     const void *fb_list, *d_small, *dyn, *grid, *Lw, *W, *picks, *slots, *ctl, *w;
+    const void *spG, *sp_tv, *sp_ts, *sp_nt, *sp_dw, *sp_sa, *fb_groups;
 };
 static_assert(sizeof(FbKey) <= sizeof(((dock_ctx*)nullptr)->fb_key), "fb_key too small");
 
-int fb_chunk(const dock_ctx* ctx, bool use_tc)
+int fb_chunk(const dock_ctx* ctx, int kind)
 {
+    const bool use_tc = kind == ENG_TC;
     const size_t ncell = (size_t)ctx->nx * ctx->ny * ctx->nz;
     const size_t budget = size_t(1) << 30;   // score grids of one chunk: <= 1 GiB
     const size_t fit = std::max<size_t>(1, budget / (ncell * sizeof(float)));
@@ -799,12 +1063,13 @@ dock_status fb_buffers(dock_ctx* ctx, int m, int ch, int k)
     TRY(ensure(ctx, ctx->fb_picks, sizeof(unsigned long long) * ch * k));
     TRY(ensure(ctx, ctx->fb_slots, sizeof(int) * ch));
     TRY(ensure(ctx, ctx->fb_ctl, sizeof(dk::FbCtl)));
+    TRY(ensure(ctx, ctx->fb_groups, sizeof(sp::Group) * ch));
     return DOCK_OK;
 }
 
 // Capture + instantiate the fallback graph for this key (ctx->stream is redirected to the private capture
 // streams while the existing launch helpers record into the graph).
-dock_status build_fb_graph(dock_ctx* ctx, const FbKey& key, const dk::FbDyn* d_dyn)
+dock_status build_fb_graph(dock_ctx* ctx, const FbKey& key, const dk::FbDyn* d_dyn, const SpCall* sc)
 {
     if (ctx->fb_exec) {
         cudaGraphExecDestroy(ctx->fb_exec);
@@ -843,12 +1108,25 @@ dock_status build_fb_graph(dock_ctx* ctx, const FbKey& key, const dk::FbDyn* d_d
         ctx->stream = cs2;
         dk::k_fb_chunk<<<1, 128, 0, cs2>>>(fb_cnt, static_cast<const int*>(ctx->fb_list.p), ctl, slots, ch);
         CU(cudaGetLastError());
-        const int nvox = (ch + dk::RB - 1) / dk::RB * dk::RB * ctx->P;
-        dk::k_voxelize_dyn<<<(nvox + 127) / 128, 128, 0, cs2>>>(&d_dyn->vox);
-        CU(cudaGetLastError());
         const float* Lw = static_cast<const float*>(ctx->fb_Lw.p);
         float* grid = static_cast<float*>(ctx->fb_grid.p);
-        if (key.use_tc) {
+        if (key.kind != ENG_SPARSE) {
+            const int nvox = (ch + dk::RB - 1) / dk::RB * dk::RB * ctx->P;
+            dk::k_voxelize_dyn<<<(nvox + 127) / 128, 128, 0, cs2>>>(&d_dyn->vox);
+            CU(cudaGetLastError());
+        }
+        if (key.kind == ENG_SPARSE) {
+            // the main pass's atom grids and term tables stay valid until the next call: one single-rotation
+            // group per flagged slot, GRID epilogue into row = chunk position
+            auto* groups = static_cast<sp::Group*>(ctx->fb_groups.p);
+            sp::k_sparse_fb_groups<<<(ch + 127) / 128, 128, 0, cs2>>>(
+                slots, &ctl->n_live, static_cast<const int*>(ctx->sp_slot_atoms.p), groups, ch);
+            CU(cudaGetLastError());
+            sp::SpArgs a = sp_args(ctx, *sc, groups, ch);
+            a.grid = grid;
+            a.n_live = &ctl->n_live;
+            CU(dock_launch_sparse(sc->xts, true, ctx->sp_tmap, sc->smem, a, (int)(ch * a.G), cs2));
+        } else if (key.kind == ENG_TC) {
             TRY(pack_weights_tc(ctx, m, key.v, ch, Lw, &ctx->fb_W));
             tc::TcArgs a = tc_args(ctx, m, key.v, ch, key.G, static_cast<const unsigned char*>(ctx->fb_W.p));
             a.grid = grid;
@@ -911,23 +1189,35 @@ dock_status build_fb_graph(dock_ctx* ctx, const FbKey& key, const dk::FbDyn* d_d
 }
 
 // Enqueue the fallback graph on the context stream (no host synchronisation).
-dock_status launch_fallback(dock_ctx* ctx, int m, bool use_tc, int v, int k, int rho, const dk::FbDyn* d_dyn)
+dock_status launch_fallback(dock_ctx* ctx, int m, int kind, int k, int rho, const dk::FbDyn* d_dyn,
+                            const SpCall* sc)
 {
-    const int ch = fb_chunk(ctx, use_tc);
+    const int ch = fb_chunk(ctx, kind);
     TRY(fb_buffers(ctx, m, ch, k));
     FbKey key;
     memset(&key, 0, sizeof(key));
     key.m = m;
-    key.use_tc = use_tc;
-    key.v = use_tc ? v : 0;
-    if (use_tc) {
+    key.kind = kind;
+    if (kind == ENG_SPARSE) {
+        key.sp_nat = sc->n_at;
+        key.sp_npl = sc->npl;
+        key.sp_smem = sc->smem;
+        key.sp_xts = sc->xts;
+        key.spG = ctx->sp_G.p;
+        key.sp_tv = ctx->sp_tv.p;
+        key.sp_ts = ctx->sp_ts.p;
+        key.sp_nt = ctx->sp_nt.p;
+        key.sp_dw = ctx->sp_dw.p;
+        key.sp_sa = ctx->sp_slot_atoms.p;
+        key.fb_groups = ctx->fb_groups.p;
+    } else if (kind == ENG_TC) {
         int vv = 0, G = 0;
         if (!plan_tc_launch(ctx, m, ch, &vv, &G)) return fail(ctx, DOCK_E_UNSUPPORTED, "no tensor-core plan");
         key.v = vv;
         key.G = G;
         const TcPlan& tp = ctx->tcplan[vv][m];
         TRY(ensure(ctx, ctx->fb_W, (size_t)tp.nsteps * tc::WCHUNK));
-    } else {
+    } else if (kind == ENG_FFMA) {
         key.G = choose_regions(ctx, (ch + dk::RB - 1) / dk::RB);
     }
     key.k = k;
@@ -949,7 +1239,7 @@ dock_status launch_fallback(dock_ctx* ctx, int m, bool use_tc, int v, int k, int
     key.ctl = ctx->fb_ctl.p;
     key.w = ctx->d_w;
     if (!ctx->fb_exec || memcmp(&key, ctx->fb_key, sizeof(key)) != 0) {
-        TRY(build_fb_graph(ctx, key, d_dyn));
+        TRY(build_fb_graph(ctx, key, d_dyn, sc));
         memcpy(ctx->fb_key, &key, sizeof(key));
     }
     CU(cudaGraphLaunch(ctx->fb_exec, ctx->stream));
@@ -1239,8 +1529,9 @@ dock_status dock_set_tuning(dock_ctx* ctx, int key, int64_t value)
             return DOCK_OK;
         case DOCK_TUNE_FORCE_FALLBACK: ctx->force_fallback = value ? 1 : 0; return DOCK_OK;
         case DOCK_TUNE_ENGINE:
-            if (value < 0 || value > 3)
-                return fail(ctx, DOCK_E_INVALID_ARG, "engine must be 0 (auto), 1 (FFMA), 2 (tcgen05) or 3 (FFT)");
+            if (value < 0 || value > 4)
+                return fail(ctx, DOCK_E_INVALID_ARG,
+                            "engine must be 0 (auto), 1 (FFMA), 2 (tcgen05), 3 (FFT) or 4 (sparse ligand)");
             ctx->engine = (int)value;
             return DOCK_OK;
         case DOCK_TUNE_TC_VARIANT:
@@ -1307,7 +1598,10 @@ dock_status dock_get_info(const dock_ctx* ctx, dock_info* info)
         info->cand_max_last = (unsigned)ctx->h_small[2];
     }
     cudaGetLastError();
-    info->fb_chunk = fb_chunk(ctx, ctx->engine_last == 2);
+    info->fb_chunk = fb_chunk(ctx, ctx->engine_last);
+    info->sp_atom_grids_last = ctx->sp_natoms_last;
+    info->sp_terms_last = ctx->sp_terms_last;
+    if (ctx->engine_last == ENG_SPARSE) info->sp_row_last = ctx->sp_tx_last;
     return DOCK_OK;
 }
 
@@ -1357,18 +1651,25 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
         TRY(ensure(ctx, ctx->poses, sizeof(dock_pose) * (size_t)n_units * k));
         d_poses = ctx->poses.p;
     }
-    // the direct engines' fallback buffers exist before staging (their addresses travel in dk::FbDyn)
-    bool use_tc = false;
+    // engine; the direct engines' fallback buffers exist before staging (their addresses travel in dk::FbDyn)
+    int kind = ENG_FFT;
+    SpCall sc;
     if (ctx->engine != 3) {
-        TRY(select_engine(ctx, m, &use_tc));
-        TRY(fb_buffers(ctx, m, fb_chunk(ctx, use_tc), k));
+        if (ctx->engine == 0 || ctx->engine == 4)
+            TRY(sp_prepare(ctx, m, probes, n_probes, n_rot, unit_begin, unit_end, &sc));
+        TRY(select_engine(ctx, m, sc.ok, sp_better(ctx, sc, m, n_units), &kind));
+        TRY(fb_buffers(ctx, m, fb_chunk(ctx, kind), k));
     }
-    dk::FbDyn fb = fb_template(ctx, m, fb_chunk(ctx, use_tc), unit_begin, n_rot, d_poses);
+    const bool use_tc = kind == ENG_TC;
+    dk::FbDyn fb = fb_template(ctx, m, fb_chunk(ctx, kind), unit_begin, n_rot, d_poses);
     const double *d_xyz, *d_rot;
     const float* d_coef;
     const int* d_off;
     const dk::FbDyn* d_fb = nullptr;
-    TRY(stage_inputs(ctx, probes, n_probes, rot, n_rot, &d_xyz, &d_coef, &d_off, &d_rot, &fb, &d_fb));
+    const void* d_groups = nullptr;
+    TRY(stage_inputs(ctx, probes, n_probes, rot, n_rot, &d_xyz, &d_coef, &d_off, &d_rot, &fb, &d_fb,
+                     kind == ENG_SPARSE ? sc.groups.data() : nullptr,
+                     kind == ENG_SPARSE ? sizeof(sp::Group) * sc.groups.size() : 0, &d_groups));
 
     unsigned int* fb_cnt = reinterpret_cast<unsigned int*>(ctx->d_small + 1);
     unsigned int* cand_max = reinterpret_cast<unsigned int*>(ctx->d_small + 2);
@@ -1379,8 +1680,11 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
     ctx->kernels_last++;
 
     // a1: voxelize (+ rotation / box validation; errors are sticky device status bits)
-    TRY(run_voxelize(ctx, m, n_units, unit_begin, nullptr, n_rot, d_xyz, d_coef, d_off, d_rot, ctx->d_w,
-                     static_cast<float*>(ctx->Lw.p)));
+    if (kind == ENG_SPARSE)
+        TRY(sp_run_pre(ctx, sc, n_units, unit_begin, n_rot, d_xyz, d_coef, d_off, d_rot, ctx->d_w));
+    else
+        TRY(run_voxelize(ctx, m, n_units, unit_begin, nullptr, n_rot, d_xyz, d_coef, d_off, d_rot, ctx->d_w,
+                         static_cast<float*>(ctx->Lw.p)));
 
     if (ctx->engine == 3) {
         // comparison engine: FFT score grids + exact greedy (no fused top-k, no fallback needed); this engine
@@ -1403,12 +1707,27 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
     auto* mup = static_cast<unsigned long long*>(ctx->mu.p);
     auto* cntp = static_cast<unsigned int*>(ctx->cnt.p);
     auto* candp = static_cast<unsigned long long*>(ctx->cand.p);
-    int v_used = 0;
-    if (use_tc) {
+    if (kind == ENG_SPARSE) {
+        const int64_t n_groups = (int64_t)sc.groups.size();
+        sp::SpArgs a = sp_args(ctx, sc, static_cast<const sp::Group*>(d_groups), n_groups);
+        a.k = k;
+        a.rho = rho;
+        a.cap = cap;
+        a.T = Tp;
+        a.mu = mup;
+        a.cnt = cntp;
+        a.cand = candp;
+        const int64_t items = n_groups * a.G;
+        if (items > 0x7fffffff) return fail(ctx, DOCK_E_UNSUPPORTED, "too many work items");
+        CU(cudaEventRecord(ctx->ev_corr[0], ctx->stream));
+        CU(dock_launch_sparse(sc.xts, false, ctx->sp_tmap, sc.smem, a, (int)items, ctx->stream));
+        CU(cudaEventRecord(ctx->ev_corr[1], ctx->stream));
+        ctx->regions_last = a.G;
+        ctx->items_last = items;
+    } else if (use_tc) {
         const int64_t n_blocks = (n_units + tc::ROT - 1) / tc::ROT;
         int v = 0, G = 0;
         if (!plan_tc_launch(ctx, m, n_units, &v, &G)) return fail(ctx, DOCK_E_UNSUPPORTED, "no tensor-core plan");
-        v_used = v;
         TRY(pack_weights_tc(ctx, m, v, n_units, static_cast<const float*>(ctx->Lw.p)));
         ctx->tc_variant_last = v;
         ctx->tc_ksteps_last = ctx->tcplan[v][m].nsteps;
@@ -1491,7 +1810,7 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
     ctx->kernels_last++;
 
     // a6': exact fallback of the flagged rotations, driven by the device-side flag count
-    TRY(launch_fallback(ctx, m, use_tc, v_used, k, rho, d_fb));
+    TRY(launch_fallback(ctx, m, kind, k, rho, d_fb, &sc));
 
     // a7: output.  Device output: return now (results and errors at dock_sync / the next sync point);
     // host output: copy back and synchronise.
@@ -1523,10 +1842,21 @@ dock_status dock_score_grid(dock_ctx* ctx, const dock_probe_desc* probe, const d
     int m = 0;
     TRY(validate_probes(ctx, probe, 1, &m));
     TRY(make_plan(ctx, m));
+    int kind = ENG_FFT;
+    SpCall sc;
+    if (ctx->engine != 3) {
+        if (ctx->engine == 0 || ctx->engine == 4) TRY(sp_prepare(ctx, m, probe, 1, 1, 0, 1, &sc));
+        TRY(select_engine(ctx, m, sc.ok, sp_better(ctx, sc, m, 1), &kind));
+    } else {
+        ctx->engine_last = 3;
+    }
     const double *d_xyz, *d_rot;
     const float* d_coef;
     const int* d_off;
-    TRY(stage_inputs(ctx, probe, 1, rot9, 1, &d_xyz, &d_coef, &d_off, &d_rot));
+    const void* d_groups = nullptr;
+    TRY(stage_inputs(ctx, probe, 1, rot9, 1, &d_xyz, &d_coef, &d_off, &d_rot, nullptr, nullptr,
+                     kind == ENG_SPARSE ? sc.groups.data() : nullptr,
+                     kind == ENG_SPARSE ? sizeof(sp::Group) * sc.groups.size() : 0, &d_groups));
     const size_t ncell = (size_t)ctx->nx * ctx->ny * ctx->nz;
     const int m3 = m * m * m;
     TRY(ensure(ctx, ctx->Lw, sizeof(float) * ctx->P * m3 * dk::RB));
@@ -1537,23 +1867,24 @@ dock_status dock_score_grid(dock_ctx* ctx, const dock_probe_desc* probe, const d
     if (need) TRY(ensure(ctx, ctx->grid, sizeof(float) * need));
     float* g_out = out_dev ? out : static_cast<float*>(ctx->grid.p);
     float* g_pt = per_term ? (pt_dev ? per_term : static_cast<float*>(ctx->grid.p) + (out_dev ? 0 : ncell)) : nullptr;
-    bool use_tc = false;
-    if (ctx->engine == 3) ctx->engine_last = 3;
-    else TRY(select_engine(ctx, m, &use_tc));
-    auto grid_fn = [&](float* dst) -> dock_status {
-        if (ctx->engine == 3) return run_grid_fft(ctx, m, 0, 1, static_cast<const float*>(ctx->Lw.p), dst);
-        return use_tc ? run_grid_tc(ctx, m, 1, static_cast<const float*>(ctx->Lw.p), dst)
-                      : run_grid(ctx, m, 1, static_cast<const float*>(ctx->Lw.p), dst);
-    };
-    TRY(run_voxelize(ctx, m, 1, 0, nullptr, 1, d_xyz, d_coef, d_off, d_rot, ctx->d_w, static_cast<float*>(ctx->Lw.p)));
-    TRY(grid_fn(g_out));
-    if (per_term) {
-        for (int p = 0; p < ctx->P; p++) {
-            TRY(run_voxelize(ctx, m, 1, 0, nullptr, 1, d_xyz, d_coef, d_off, d_rot, ctx->d_eye + (size_t)p * ctx->P,
-                             static_cast<float*>(ctx->Lw.p)));
-            TRY(grid_fn(g_pt + ncell * p));
+    // one score grid with weights w (folded into L, or into the atom grids of the sparse engine)
+    auto grid_fn = [&](const float* w, float* dst) -> dock_status {
+        if (kind == ENG_SPARSE) {
+            TRY(sp_run_pre(ctx, sc, 1, 0, 1, d_xyz, d_coef, d_off, d_rot, w));
+            sp::SpArgs a = sp_args(ctx, sc, static_cast<const sp::Group*>(d_groups), 1);
+            a.grid = dst;
+            CU(dock_launch_sparse(sc.xts, true, ctx->sp_tmap, sc.smem, a, a.G, ctx->stream));
+            ctx->kernels_last++;
+            return DOCK_OK;
         }
-    }
+        TRY(run_voxelize(ctx, m, 1, 0, nullptr, 1, d_xyz, d_coef, d_off, d_rot, w, static_cast<float*>(ctx->Lw.p)));
+        if (kind == ENG_FFT) return run_grid_fft(ctx, m, 0, 1, static_cast<const float*>(ctx->Lw.p), dst);
+        return kind == ENG_TC ? run_grid_tc(ctx, m, 1, static_cast<const float*>(ctx->Lw.p), dst)
+                              : run_grid(ctx, m, 1, static_cast<const float*>(ctx->Lw.p), dst);
+    };
+    TRY(grid_fn(ctx->d_w, g_out));
+    if (per_term)
+        for (int p = 0; p < ctx->P; p++) TRY(grid_fn(ctx->d_eye + (size_t)p * ctx->P, g_pt + ncell * p));
     if (!out_dev) CU(cudaMemcpyAsync(out, g_out, sizeof(float) * ncell, cudaMemcpyDeviceToHost, ctx->stream));
     if (per_term && !pt_dev)
         CU(cudaMemcpyAsync(per_term, g_pt, sizeof(float) * ncell * ctx->P, cudaMemcpyDeviceToHost, ctx->stream));

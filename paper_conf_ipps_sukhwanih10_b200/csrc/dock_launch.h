@@ -7,6 +7,7 @@
 
 #include "dock_kernels.cuh"
 #include "dock_tc.cuh"
+#include "dock_sparse.cuh"
 
 // FP32 FFMA engine k_corr<m, grid>
 cudaError_t dock_launch_ffma(int m, bool grid, const CUtensorMap& tmap, int smem, const dk::CorrArgs& a, int nblocks,
@@ -21,6 +22,24 @@ cudaError_t dock_launch_tcs128(int m, bool grid, const CUtensorMap& tmap, const 
                                const tc::TcArgs& a, int nblocks, cudaStream_t st);
 cudaError_t dock_launch_tcs160(int m, bool grid, const CUtensorMap& tmap, const CUtensorMap& tmap_pair, int smem,
                                const tc::TcArgs& a, int nblocks, cudaStream_t st);
+
+// sparse-ligand engine k_corr_sparse<xts, grid> (dock_sparse.cuh); xts = translations per lane along x
+cudaError_t dock_launch_sparse2(bool grid, const CUtensorMap& gmap, int smem, const sp::SpArgs& a, int nblocks,
+                                cudaStream_t st);
+cudaError_t dock_launch_sparse4(bool grid, const CUtensorMap& gmap, int smem, const sp::SpArgs& a, int nblocks,
+                                cudaStream_t st);
+cudaError_t dock_launch_sparse5(bool grid, const CUtensorMap& gmap, int smem, const sp::SpArgs& a, int nblocks,
+                                cudaStream_t st);
+inline cudaError_t dock_launch_sparse(int xts, bool grid, const CUtensorMap& gmap, int smem, const sp::SpArgs& a,
+                                      int nblocks, cudaStream_t st)
+{
+    switch (xts) {
+        case 2: return dock_launch_sparse2(grid, gmap, smem, a, nblocks, st);
+        case 4: return dock_launch_sparse4(grid, gmap, smem, a, nblocks, st);
+        case 5: return dock_launch_sparse5(grid, gmap, smem, a, nblocks, st);
+        default: return cudaErrorInvalidValue;
+    }
+}
 
 // rows per tile of the streamed kernel for a row width: Q * NTT <= 512 TMEM columns
 constexpr int tcs_q(int ntt) { return ntt == 64 ? 8 : ntt == 160 ? 3 : 4; }

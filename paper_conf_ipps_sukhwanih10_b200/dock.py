@@ -97,6 +97,10 @@ def dock_init(receptor, weights, spacing: float = 0.8, m_max: int = 8, device: i
         sh = stream
     else:
         sh = stream.cuda_stream
+    if sh == 0:
+        # torch's default stream is the legacy default stream: pass cudaStreamLegacy (a NULL stream asks the
+        # library to create a private one, which torch's work would not be ordered with)
+        sh = 1
     rp, rk = _buf(receptor, "f4")
     wp, wk = _buf(weights, "f4")
     g = N.dock_grid_desc(nx, ny, nz, P, m_max, device, float(spacing), C.c_void_p(sh))

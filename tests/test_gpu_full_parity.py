@@ -26,7 +26,7 @@ import oracle_cache  # noqa: E402  (input generation + hash only; no arithmetic 
 
 pytestmark = pytest.mark.gpu
 H = g.SPACING
-ENGINES = [1, 2, 3]   # 1 FP32 FFMA, 2 tcgen05 variant 1, 3 tcgen05 variant 2
+ENGINES = [1, 2, 3, 4]   # 1 FP32 FFMA, 2 tcgen05 variant 1, 3 tcgen05 variant 2, 4 sparse ligand
 
 
 @pytest.fixture(scope="module")
@@ -60,8 +60,8 @@ def test_full_workload_parity(D, orc, cfg, engine):
     assert (ref["status"] == 0).all()
     dev = torch.device("cuda", 0)
     ctx = D.dock_init(torch.from_numpy(R).to(dev), torch.from_numpy(w).to(dev), H, m_max=c.m, device=0)
-    D.dock_set_tuning(ctx, D.DOCK_TUNE_ENGINE, 1 if engine == 1 else 2)
-    if engine >= 2:
+    D.dock_set_tuning(ctx, D.DOCK_TUNE_ENGINE, {1: 1, 2: 2, 3: 2, 4: 4}[engine])
+    if engine in (2, 3):
         D.dock_set_tuning(ctx, D.DOCK_TUNE_TC_VARIANT, engine - 1)
     n = c.n_probes * c.n_rot
     dprobes = [{"xyz": torch.from_numpy(p.xyz).to(dev), "coef": torch.from_numpy(p.coef).to(dev), "m": p.m}
@@ -71,7 +71,7 @@ def test_full_workload_parity(D, orc, cfg, engine):
     torch.cuda.synchronize()
     info = D.dock_get_info(ctx)
     ctx.close()
-    eng = 1 if info["engine_last"] == 1 else 1 + info["tc_variant_last"]
+    eng = {1: 1, 4: 4}.get(info["engine_last"], 1 + info["tc_variant_last"])
     assert eng == engine
     poses = D.poses_from_device(out)
     assert (poses["rot"] == np.arange(n)[:, None] % c.n_rot).all()

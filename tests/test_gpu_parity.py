@@ -28,21 +28,24 @@ def D():
 
 # engine ids used by the tests: 1 = FP32 FFMA; 2 = tcgen05 variant 1 (one channel group, resident receptor
 # boxes, 128 translations x 4 rows); 3 = tcgen05 variant 2 (receptor streamed per (channel group, z-plane),
-# any P, 64 / 128 / 160 translations per row).  A tcgen05 variant that cannot run a case runs the other one.
-ENGINES = [1, 2, 3]
+# any P, 64 / 128 / 160 translations per row); 4 = sparse ligand (FP32 gathers of per-atom channel grids at
+# the occupied voxels, NEXT-3).  A tcgen05 variant that cannot run a case runs the other one.
+ENGINES = [1, 2, 3, 4]
 
 
 def _ctx(D, R, w, m_max, engine=0):
     ctx = D.dock_init(R, w, H, m_max=m_max)
+    ctx.test_engine = engine
     if engine:
-        D.dock_set_tuning(ctx, D.DOCK_TUNE_ENGINE, 1 if engine == 1 else 2)
-        if engine >= 2:
+        D.dock_set_tuning(ctx, D.DOCK_TUNE_ENGINE, {1: 1, 2: 2, 3: 2, 4: 4}[engine])
+        if engine in (2, 3):
             D.dock_set_tuning(ctx, D.DOCK_TUNE_TC_VARIANT, engine - 1)
     return ctx
 
 
 def _engine_id(info):
-    return 1 if info["engine_last"] == 1 else 1 + info["tc_variant_last"]
+    e = info["engine_last"]
+    return {1: 1, 4: 4}.get(e, 1 + info["tc_variant_last"])
 
 
 def _oracle_SA(orc, R, w, pr, q):
@@ -186,7 +189,7 @@ def test_score_grid_within_tolerance(D, orc, shape, m, P, kind, engine):
     ctx.close()
 
 
-@pytest.mark.parametrize("engine", [1])   # bf16x3 is exact only to ~2^-24 relative: FFMA engine
+@pytest.mark.parametrize("engine", [1, 4])   # bf16x3 is exact only to ~2^-24 relative: FFMA and sparse engines
 def test_delta_probe_bitwise(D, engine):
     """P4: one atom at the centre, m = 1, coef = e_p -> S == R_p bitwise on the GPU."""
     P = 3
@@ -200,7 +203,7 @@ def test_delta_probe_bitwise(D, engine):
     ctx.close()
 
 
-@pytest.mark.parametrize("engine", [1])
+@pytest.mark.parametrize("engine", [1, 4])
 def test_shift_equivariance_bitwise(D, engine):
     """P5: single atom on voxel v0 -> S = roll(R, -v0) bitwise."""
     R = g.receptor_uniform((24, 20, 16), 1)
@@ -315,8 +318,10 @@ def test_fallback_path_identical(D, engine):
 
 @pytest.mark.parametrize("engine", ENGINES)
 def test_invariance_batch_shard_launch(D, engine):
-    """Per-rotation results are bitwise independent of batch position, batch size,
-    regions per batch (launch configuration), candidate cap and shard range."""
+    """Per-rotation results (rotation, t_lin and score bits) are bitwise independent of batch position, batch
+    size, regions per batch (launch configuration), candidate cap and shard range.  The DOCK_POSE_FALLBACK
+    flag only records which path produced a pose (the candidate lists or the exact fallback, whose score
+    bits are the same), and that may depend on the launch configuration."""
     P, m = 4, 4
     R = g.receptor_ftmap_like((64, 48, 40), P)
     w = g.weights(P)
@@ -325,12 +330,16 @@ def test_invariance_batch_shard_launch(D, engine):
     ctx = _ctx(D, R, w, m, engine)
     ref = D.dock_probe_batch(ctx, probes, rot, k=4, rho=1)
     n = len(probes) * len(rot)
+    def same(a, b):
+        return all(np.array_equal(a[f].view(np.uint32) if f == "score" else a[f],
+                                  b[f].view(np.uint32) if f == "score" else b[f]) for f in ("rot", "t_lin", "score"))
+
     for b, e in [(0, 5), (5, 31), (31, n), (7, 8)]:
         part = D.dock_probe_batch(ctx, probes, rot, unit_begin=b, unit_end=e, k=4, rho=1)
-        assert np.array_equal(part, ref[b:e])
+        assert same(part, ref[b:e])
     for G in (1, 3, 7):
         D.dock_set_tuning(ctx, D.DOCK_TUNE_REGIONS, G)
-        assert np.array_equal(D.dock_probe_batch(ctx, probes, rot, k=4, rho=1), ref)
+        assert same(D.dock_probe_batch(ctx, probes, rot, k=4, rho=1), ref)
     D.dock_set_tuning(ctx, D.DOCK_TUNE_REGIONS, 0)
     D.dock_set_tuning(ctx, D.DOCK_TUNE_CAND_CAP, 32)   # small cap: overflowing rotations take the fallback
     capped = D.dock_probe_batch(ctx, probes, rot, k=4, rho=1)
@@ -515,7 +524,7 @@ def test_prod_config_sampled(D, orc, engine):
     assert info["fallback_last"] <= 80 and _engine_id(info) == engine
 
 
-@pytest.mark.parametrize("engine", [1, 3])
+@pytest.mark.parametrize("engine", [1, 3, 4])
 def test_large_config_sampled(D, orc, engine):
     """configs[4] shape: 160^3 receptor, 8^3 probe, 22 terms (pairwise-potential channels), k=4, rho=1.
     A 256-rotation slice of the 70k-rotation set is docked on the GPU (FFMA engine, and tcgen05 variant 2:
@@ -545,7 +554,7 @@ def test_max_terms_probe_and_k(D, orc, engine, rho):
     probes = g.probes(1, m, P)
     rot = g.rotations(5, with_cube_group=False)
     poses, info, _ = _dock_and_validate(D, orc, R, w, probes, rot, k, rho, engine=engine)
-    assert _engine_id(info) == (1 if engine == 1 else 3)   # 8 channel groups: tcgen05 variant 2
+    assert _engine_id(info) == {1: 1, 4: 4}.get(engine, 3)   # 8 channel groups: tcgen05 variant 2
     ctx = _ctx(D, R, w, m, engine)
     S_g = D.dock_score_grid(ctx, probes[0], rot[1])
     ctx.close()
