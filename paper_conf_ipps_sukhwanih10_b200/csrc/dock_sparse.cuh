@@ -417,20 +417,22 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
                 // a single-atom voxel, 0 for an absent or multi-atom term: fma(1, g, acc) == acc + g exactly);
                 // term 0 initialises the accumulators
                 float acc[RB][XTS];
+                if (tmax > 0) {
 #pragma unroll
-                for (int r = 0; r < RB; r++) {
-                    if (tmax == 0) {   // a probe without atoms scores 0 everywhere
+                    for (int r = 0; r < RB; r++) {
+                        const int4 term = s_term[r];
+                        uint32_t zo = zoff + static_cast<uint32_t>(term.y);
+                        zo = zo >= ring_bytes ? zo - ring_bytes : zo;
+                        const uint32_t ad = lane_base + zo + static_cast<uint32_t>(term.x);
+                        const float wt = __int_as_float(term.z);
+#pragma unroll
+                        for (int i = 0; i < XTS; i++) acc[r][i] = wt * lds_f32(ad + 128u * i);
+                    }
+                } else {   // a probe without atoms scores 0 everywhere
+#pragma unroll
+                    for (int r = 0; r < RB; r++)
 #pragma unroll
                         for (int i = 0; i < XTS; i++) acc[r][i] = 0.0f;
-                        continue;
-                    }
-                    const int4 term = s_term[r];
-                    uint32_t zo = zoff + static_cast<uint32_t>(term.y);
-                    zo = zo >= ring_bytes ? zo - ring_bytes : zo;
-                    const uint32_t ad = lane_base + zo + static_cast<uint32_t>(term.x);
-                    const float wt = __int_as_float(term.z);
-#pragma unroll
-                    for (int i = 0; i < XTS; i++) acc[r][i] = wt * lds_f32(ad + 128u * i);
                 }
 #pragma unroll 1
                 for (int t = 1; t < tmax; t++) {
