@@ -343,3 +343,53 @@ CONFIGS = {
     "prod": Config("prod", (128, 128, 128), 4, 4, 500, 16, 4),
     "large": Config("large", (160, 160, 160), 8, 22, 70000, 1, 4),
 }
+
+
+# --------------------------------------------------------------------------- energy minimisation (NEXT-4)
+
+
+@dataclass
+class EmSystem:
+    """Synthetic non-bonded system of FTMap's energy minimisation (§II.B; parameters are synthetic:
+    the paper gives none and CHARMM parameters are out of scope).  Pairs i < j within rc of the reference
+    coordinates (the neighbour list the paper keeps fixed over many iterations)."""
+    x0: np.ndarray      # [n][3] reference coordinates (A)
+    q: np.ndarray       # [n] charges (e)
+    R: np.ndarray       # [n] intrinsic radii (A)
+    V: np.ndarray       # [n] solute volumes (A^3)
+    eps: np.ndarray     # [n] vdW well depths
+    rm: np.ndarray      # [n] vdW radii (rm_i; rm_ij = (rm_i + rm_j)/2)
+    type: np.ndarray    # [n] atom types
+    omega: np.ndarray   # [T][T] ACE Gaussian heights (ordered type pair)
+    sigma: np.ndarray   # [T][T] ACE Gaussian widths
+    mu: np.ndarray      # [T][T] ACE atom-atom parameters
+    pairs: np.ndarray   # [n_pairs][2] int32, i < j, sorted by (i, j)
+    eps_s: float = 80.0
+    rc: float = 9.0
+
+
+def em_system(n_atoms: int = 2200, seed: int = 5001, rc: float = 9.0, spacing: float = 2.7) -> EmSystem:
+    """~n_atoms atoms on a jittered cubic lattice (min separation > 2 A) inside a sphere (protein-like density)."""
+    rng = np.random.default_rng(seed)
+    side = int(np.ceil((n_atoms * 6.0 / np.pi) ** (1.0 / 3.0))) + 2
+    g = np.arange(side) * spacing
+    pts = np.stack(np.meshgrid(g, g, g, indexing="ij"), -1).reshape(-1, 3)
+    c = pts.mean(0)
+    pts = pts[np.argsort(np.linalg.norm(pts - c, axis=1), kind="stable")[:n_atoms]]
+    x0 = pts + rng.uniform(-0.3, 0.3, size=pts.shape)
+    T = 6
+    typ = rng.integers(0, T, size=n_atoms).astype(np.int32)
+    d = np.linalg.norm(x0[:, None, :] - x0[None, :, :], axis=2)
+    i, j = np.nonzero(np.triu(d < rc, k=1))
+    pairs = np.stack([i, j], 1).astype(np.int32)
+    return EmSystem(x0=x0, q=rng.uniform(-0.5, 0.5, n_atoms), R=rng.uniform(1.4, 2.0, n_atoms),
+                    V=rng.uniform(10.0, 30.0, n_atoms), eps=rng.uniform(0.05, 0.2, n_atoms),
+                    rm=rng.uniform(1.7, 2.2, n_atoms), type=typ, omega=rng.uniform(0.0, 0.02, (T, T)),
+                    sigma=rng.uniform(2.5, 4.0, (T, T)), mu=rng.uniform(1.5, 3.0, (T, T)), pairs=pairs, rc=rc)
+
+
+def em_conformations(s: EmSystem, n_conf: int, seed: int = 5002, jitter: float = 0.05) -> np.ndarray:
+    """n_conf conformations [n_conf][n][3]: the reference plus small Gaussian displacements (minimisation
+    moves atoms by small amounts)."""
+    rng = np.random.default_rng(seed)
+    return s.x0[None] + rng.normal(0.0, jitter, size=(n_conf,) + s.x0.shape)

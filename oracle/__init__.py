@@ -13,3 +13,4 @@ from .oracle import (  # noqa: F401
     build_oracle, check_rotation, voxelize, score_grid, filter_greedy, dock,
     max_threads, OracleError,
 )
+from .em import build_em_oracle, em_eval  # noqa: F401  (EM non-bonded energy, NEXT-4)
