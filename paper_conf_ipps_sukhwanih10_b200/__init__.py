@@ -14,3 +14,4 @@ from ._native import (  # noqa: F401
     DOCK_TUNE_FORCE_FALLBACK, DOCK_TUNE_REGIONS, EXPORTS, LIB_PATH,
 )
 from . import parallel  # noqa: F401,E402
+from . import em  # noqa: F401,E402  (energy-minimisation non-bonded kernels, NEXT-4)

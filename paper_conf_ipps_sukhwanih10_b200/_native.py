@@ -59,7 +59,19 @@ class dock_info(C.Structure):
 
 
 EXPORTS = ["dock_init", "dock_probe", "dock_probe_batch", "dock_sync", "dock_score_grid", "dock_voxelize",
-           "dock_set_tuning", "dock_get_info", "dock_destroy", "dock_status_string", "dock_last_error"]
+           "dock_set_tuning", "dock_get_info", "dock_destroy", "dock_status_string", "dock_last_error",
+           "dock_em_init", "dock_em_eval", "dock_em_last_ms", "dock_em_destroy", "dock_em_last_error"]
+
+
+class dock_em_desc(C.Structure):
+    _fields_ = [("n_atoms", C.c_int), ("n_pairs", C.c_int), ("n_types", C.c_int), ("device", C.c_int),
+                ("eps_s", C.c_double), ("rc", C.c_double), ("stream", C.c_void_p)]
+
+
+class dock_em_params(C.Structure):
+    _fields_ = [("q", C.c_void_p), ("R", C.c_void_p), ("V", C.c_void_p), ("eps", C.c_void_p), ("rm", C.c_void_p),
+                ("type", C.c_void_p), ("omega", C.c_void_p), ("sigma", C.c_void_p), ("mu", C.c_void_p),
+                ("pairs", C.c_void_p)]
 
 _lib = None
 
@@ -87,6 +99,16 @@ def lib() -> C.CDLL:
     L.dock_status_string.restype = C.c_char_p
     L.dock_last_error.argtypes = [vp]
     L.dock_last_error.restype = C.c_char_p
+    L.dock_em_init.argtypes = [C.POINTER(dock_em_desc), C.POINTER(dock_em_params), C.POINTER(vp)]
+    L.dock_em_eval.argtypes = [vp, vp, i, vp, vp]
+    L.dock_em_last_ms.argtypes = [vp]
+    L.dock_em_last_ms.restype = C.c_double
+    L.dock_em_destroy.argtypes = [vp]
+    L.dock_em_destroy.restype = None
+    L.dock_em_last_error.argtypes = [vp]
+    L.dock_em_last_error.restype = C.c_char_p
+    L.dock_em_init.restype = C.c_int
+    L.dock_em_eval.restype = C.c_int
     for name in ("dock_init", "dock_probe", "dock_probe_batch", "dock_sync", "dock_score_grid", "dock_voxelize",
                  "dock_set_tuning", "dock_get_info"):
         getattr(L, name).restype = C.c_int

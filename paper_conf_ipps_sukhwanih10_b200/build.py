@@ -13,9 +13,9 @@ LIB = os.path.join(PKG, "libdock.so")
 # dock.cu = host logic + small kernels; launch_*.cu = one correlation-kernel family each (compiled in
 # parallel, then linked into one shared library)
 SOURCES = [os.path.join(CSRC, "dock.cu")] + sorted(glob.glob(os.path.join(CSRC, "launch_*.cu"))) + \
-    [os.path.join(CSRC, "fft_engine.cu")]
+    [os.path.join(CSRC, "fft_engine.cu"), os.path.join(CSRC, "em.cu")]
 HEADERS = (sorted(glob.glob(os.path.join(CSRC, "*.cuh"))) + sorted(glob.glob(os.path.join(CSRC, "*.h"))) +
-           [os.path.join(ROOT, "include", "dock.h")])
+           sorted(glob.glob(os.path.join(ROOT, "include", "*.h"))))
 
 NVCC_FLAGS = [
     "-gencode", "arch=compute_100a,code=sm_100a",

@@ -18,7 +18,8 @@ def lib():
 
 
 def _header_functions():
-    src = open(os.path.join(ROOT, "include", "dock.h")).read()
+    import glob
+    src = "".join(open(h).read() for h in sorted(glob.glob(os.path.join(ROOT, "include", "*.h"))))
     src = re.sub(r"/\*.*?\*/", "", src, flags=re.S)
     return sorted(set(re.findall(r"\b(dock_[a-z_]+)\s*\(", src)))
 
@@ -62,8 +63,10 @@ def test_struct_layouts_match_header(tmp_path):
     if not cc:
         pytest.skip("no C compiler")
     structs = {"dock_pose": N.dock_pose, "dock_grid_desc": N.dock_grid_desc,
-               "dock_probe_desc": N.dock_probe_desc, "dock_info": N.dock_info}
-    lines = ['#include <stdio.h>', '#include <stddef.h>', '#include "dock.h"', "int main(void) {"]
+               "dock_probe_desc": N.dock_probe_desc, "dock_info": N.dock_info, "dock_em_desc": N.dock_em_desc,
+               "dock_em_params": N.dock_em_params}
+    lines = ['#include <stdio.h>', '#include <stddef.h>', '#include "dock.h"', '#include "dock_em.h"',
+             "int main(void) {"]
     for name, cls in structs.items():
         lines.append(f'printf("{name} size %zu\\n", sizeof({name}));')
         for f, _ in cls._fields_:
