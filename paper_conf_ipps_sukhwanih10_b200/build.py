@@ -32,8 +32,23 @@ def _nvcc() -> str:
     return "nvcc"
 
 
+STAMP = os.path.join(PKG, "libdock.defs")   # the DOCK_NVCC_DEFS the library was built with
+
+
+def _defs() -> str:
+    return " ".join(os.environ.get("DOCK_NVCC_DEFS", "").split())
+
+
 def stale() -> bool:
+    """Rebuild when a source is newer than the library, or when the experiment defines (DOCK_NVCC_DEFS)
+    differ from those the library was built with (a tuning build is never silently reused)."""
     if not os.path.exists(LIB):
+        return True
+    try:
+        with open(STAMP) as f:
+            if f.read().strip() != _defs():
+                return True
+    except OSError:
         return True
     t = os.path.getmtime(LIB)
     return any(os.path.getmtime(p) > t for p in SOURCES + HEADERS)
@@ -75,6 +90,8 @@ def build_native(force: bool = False, verbose: bool = False) -> str:
     with open(os.path.join(PKG, "libdock.ptxas.txt"), "w") as f:
         f.write(log)
     os.replace(tmp, LIB)
+    with open(STAMP, "w") as f:
+        f.write(_defs() + "\n")
     return LIB
 
 

@@ -8,9 +8,6 @@ G='"value": [0-9.]*\|"launch_ms": [0-9.]*\|"executed_frac": [0-9.]*\|fallback_ro
 echo "== V1"; timeout 300 $B --tc-variant 1 > gpurun_out/tc_${TAG}_q4.log 2>&1; grep -o "$G" gpurun_out/tc_${TAG}_q4.log
 echo "== V1 epi8"; timeout 300 $B --tc-variant 1 --tc-epi 8 > gpurun_out/tc_${TAG}_e8.log 2>&1; grep -o "$G" gpurun_out/tc_${TAG}_e8.log
 echo "== V2"; timeout 300 $B --tc-variant 2 > gpurun_out/tc_${TAG}_q2.log 2>&1; grep -o "$G" gpurun_out/tc_${TAG}_q2.log
-echo "== V3"; timeout 300 $B --tc-variant 3 > gpurun_out/tc_${TAG}_v3.log 2>&1; grep -o "$G" gpurun_out/tc_${TAG}_v3.log
-echo "== V4"; timeout 300 $B --tc-variant 4 > gpurun_out/tc_${TAG}_v4.log 2>&1; grep -o "$G" gpurun_out/tc_${TAG}_v4.log
-echo "== V4 epi4"; timeout 300 $B --tc-variant 4 --tc-epi 4 > gpurun_out/tc_${TAG}_v4e4.log 2>&1; grep -o "$G" gpurun_out/tc_${TAG}_v4e4.log
 echo "== FFMA"; timeout 300 python bench.py --steps 3 --warmup 2 --no-e2e --no-cpu-baseline --no-alt --engine ffma > gpurun_out/ffma_${TAG}.log 2>&1; grep -o '"value": [0-9.]*\|"launch_ms": [0-9.]*\|"frac": [0-9.]*' gpurun_out/ffma_${TAG}.log
 if [ "${NCU:-1}" = "1" ]; then
 timeout 900 ncu --set full --clock-control none --import-source on -k regex:${KRE:-k_corr_tc} -s 1 -c 1 \
