@@ -236,7 +236,8 @@ def roofline(pk, pk_kind, info, c, flops_launch, corr_ms, ms_step, units_local):
         gbytes = 4.0 * float(info["sp_terms_last"]) * ncell
         ach = gbytes / (corr_ms / 1000.0) / 1e9
         peak = n_sms * 128 * sm_max * 1e6 / 1e9
-        return {"bound": "smem", "engine": "sparse ligand (fp32 gathers)", "kernel": "k_corr_sparse",
+        xts = max(1, int(info.get("sp_row_last", 128)) // 32)
+        return {"bound": "smem", "engine": "sparse ligand (fp32 gathers)", "kernel": f"k_corr_sparse<{xts},false>",
                 "achieved": ach, "peak": peak, "unit": "GB/s", "frac": ach / peak, "traffic": None,
                 "peak_source": f"{n_sms} SMs x 128 B/clk shared-memory loads x {sm_max:.0f} MHz (sm_max_mhz, "
                                f"MEASURED_PEAKS.json: {pk_kind})",

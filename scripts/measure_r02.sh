@@ -1,0 +1,17 @@
+#!/bin/bash
+# Round-2 evidence (run under gpurun, 1 GPU): bench lines (prod = the headline, c64, the large config's
+# per-rank shard), the ncu launch list of the prod bench command, and one ncu --set full capture of the
+# dominant kernel of prod (k_corr_tc) and of the large shard (k_corr_sparse).
+set -u
+mkdir -p gpurun_out
+TAG=${1:-r02}
+python -c "import __graft_entry__ as e; e.build()" > gpurun_out/build_${TAG}.log 2>&1 || { tail gpurun_out/build_${TAG}.log; exit 1; }
+echo "== bench prod"; timeout 900 python bench.py > gpurun_out/bench_${TAG}_prod.json 2> gpurun_out/bench_${TAG}_prod.err; echo "rc=$?"
+echo "== bench c64"; timeout 600 python bench.py --config c64 --no-cpu-baseline > gpurun_out/bench_${TAG}_c64.json 2> gpurun_out/bench_${TAG}_c64.err; echo "rc=$?"
+echo "== bench large shard"; timeout 900 python bench.py --config large --rotations 8750 --steps 3 --warmup 3 --no-cpu-baseline --no-e2e > gpurun_out/bench_${TAG}_large.json 2> gpurun_out/bench_${TAG}_large.err; echo "rc=$?"
+echo "== launch list prod"
+timeout 900 ncu --metrics gpu__time_duration.sum --clock-control none --csv --log-file gpurun_out/launches_${TAG}_prod.csv \
+    python bench.py --steps 2 --warmup 1 --no-e2e --no-cpu-baseline --no-alt > gpurun_out/launches_${TAG}_prod.log 2>&1; echo "rc=$?"
+echo "== full capture k_corr_tc (prod)"; SKIP=1 bash scripts/ncu_kernel.sh ${TAG}_prod_tc k_corr_tc --config prod --engine tc
+echo "== full capture k_corr_sparse (large, 512 rotations)"; SKIP=1 bash scripts/ncu_kernel.sh ${TAG}_large_sparse k_corr_sparse --config large --rotations 512 --engine sparse
+ls gpurun_out | head -50
