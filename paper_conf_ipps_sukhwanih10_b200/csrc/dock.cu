@@ -726,10 +726,10 @@ dock_status make_sp_plan(dock_ctx* ctx, int m, int xts)
 
 // Plane-ring depth for tmax atoms: as deep as shared memory allows (<= NPLMAX planes: the steps beyond the
 // window m + PZ - 1 are TMA prefetch), at least the window; 0 when not even that fits.
-int sp_npl(const SpPlan& pl, int m, int tmax)
+int sp_npl(const SpPlan& pl, int m, int tmax, int zt)
 {
     const int budget = kSmemLimit - 22 * 1024;   // static shared memory of k_corr_sparse: ~20 KB (lists, terms)
-    for (int npl = sp::NPLMAX; npl >= m + sp::PZ - 1; npl--)
+    for (int npl = sp::NPLMAX; npl >= m + sp::NPG * zt - 1; npl--)
         if ((size_t)std::max(tmax, 1) * npl * pl.slot_words * 4 <= (size_t)budget) return npl;
     return 0;
 }
@@ -737,6 +737,7 @@ int sp_npl(const SpPlan& pl, int m, int tmax)
 struct SpCall {   // one sparse-engine launch over the units of a call
     bool ok = false;
     int xts = 0;                      // translations per lane along x (row width 32 * xts)
+    int zt = 1;                       // planes per warp and step
     int m = 0, tmax = 0, n_at = 0, atom_lo = 0, npl = 0, smem = 0;
     double terms = 0;                 // estimated occupied voxels summed over the units (cost model)
     std::vector<sp::Group> groups;    // rotation groups (<= sp::RB rotations of one probe)
@@ -761,15 +762,18 @@ dock_status sp_prepare(dock_ctx* ctx, int m, const dock_probe_desc* probes, int 
     if (tmax > sp::TMAX) return DOCK_OK;
     // row width: the fewest wasted x translations whose plane ring fits shared memory for tmax atoms
     // (ties: 128, then 160, then 64 translations per row)
-    int xts = 0, npl = 0, best_w = 1 << 30;
+    int xts = 0, npl = 0, zt = 1, best_w = 1 << 30;
     for (int x : {4, 5, 2}) {
         if (make_sp_plan(ctx, m, x) != DOCK_OK) continue;
-        const int n = sp_npl(ctx->spplan[m][x], m, tmax);
+        // 64-translation rows: two planes per warp and step when the ring fits, else one
+        int z = x == 2 ? 2 : 1, n = sp_npl(ctx->spplan[m][x], m, tmax, z);
+        if (!n && z == 2) n = sp_npl(ctx->spplan[m][x], m, tmax, z = 1);
         const int w = (ctx->nx + 32 * x - 1) / (32 * x) * (32 * x);
         if (n && w < best_w) {
             best_w = w;
             xts = x;
             npl = n;
+            zt = z;
         }
     }
     cudaGetLastError();
@@ -777,6 +781,7 @@ dock_status sp_prepare(dock_ctx* ctx, int m, const dock_probe_desc* probes, int 
     if (!xts) return DOCK_OK;   // ineligible, not an error
     const SpPlan& pl = ctx->spplan[m][xts];
     sc->xts = xts;
+    sc->zt = zt;
     int off = 0;
     for (int p = 0; p < p_lo; p++) off += probes[p].n_atoms;
     sc->m = m;
@@ -1125,7 +1130,7 @@ dock_status build_fb_graph(dock_ctx* ctx, const FbKey& key, const dk::FbDyn* d_d
             sp::SpArgs a = sp_args(ctx, *sc, groups, ch);
             a.grid = grid;
             a.n_live = &ctl->n_live;
-            CU(dock_launch_sparse(sc->xts, true, ctx->sp_tmap, sc->smem, a, (int)(ch * a.G), cs2));
+            CU(dock_launch_sparse(sc->xts, sc->zt, true, ctx->sp_tmap, sc->smem, a, (int)(ch * a.G), cs2));
         } else if (key.kind == ENG_TC) {
             TRY(pack_weights_tc(ctx, m, key.v, ch, Lw, &ctx->fb_W));
             tc::TcArgs a = tc_args(ctx, m, key.v, ch, key.G, static_cast<const unsigned char*>(ctx->fb_W.p));
@@ -1202,7 +1207,7 @@ dock_status launch_fallback(dock_ctx* ctx, int m, int kind, int k, int rho, cons
         key.sp_nat = sc->n_at;
         key.sp_npl = sc->npl;
         key.sp_smem = sc->smem;
-        key.sp_xts = sc->xts;
+        key.sp_xts = sc->xts * 8 + sc->zt;
         key.spG = ctx->sp_G.p;
         key.sp_tv = ctx->sp_tv.p;
         key.sp_ts = ctx->sp_ts.p;
@@ -1720,7 +1725,7 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
         const int64_t items = n_groups * a.G;
         if (items > 0x7fffffff) return fail(ctx, DOCK_E_UNSUPPORTED, "too many work items");
         CU(cudaEventRecord(ctx->ev_corr[0], ctx->stream));
-        CU(dock_launch_sparse(sc.xts, false, ctx->sp_tmap, sc.smem, a, (int)items, ctx->stream));
+        CU(dock_launch_sparse(sc.xts, sc.zt, false, ctx->sp_tmap, sc.smem, a, (int)items, ctx->stream));
         CU(cudaEventRecord(ctx->ev_corr[1], ctx->stream));
         ctx->regions_last = a.G;
         ctx->items_last = items;
@@ -1873,7 +1878,7 @@ dock_status dock_score_grid(dock_ctx* ctx, const dock_probe_desc* probe, const d
             TRY(sp_run_pre(ctx, sc, 1, 0, 1, d_xyz, d_coef, d_off, d_rot, w));
             sp::SpArgs a = sp_args(ctx, sc, static_cast<const sp::Group*>(d_groups), 1);
             a.grid = dst;
-            CU(dock_launch_sparse(sc.xts, true, ctx->sp_tmap, sc.smem, a, a.G, ctx->stream));
+            CU(dock_launch_sparse(sc.xts, sc.zt, true, ctx->sp_tmap, sc.smem, a, a.G, ctx->stream));
             ctx->kernels_last++;
             return DOCK_OK;
         }

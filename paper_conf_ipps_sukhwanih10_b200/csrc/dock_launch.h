@@ -23,20 +23,20 @@ cudaError_t dock_launch_tcs128(int m, bool grid, const CUtensorMap& tmap, const 
 cudaError_t dock_launch_tcs160(int m, bool grid, const CUtensorMap& tmap, const CUtensorMap& tmap_pair, int smem,
                                const tc::TcArgs& a, int nblocks, cudaStream_t st);
 
-// sparse-ligand engine k_corr_sparse<xts, grid> (dock_sparse.cuh); xts = translations per lane along x
-cudaError_t dock_launch_sparse2(bool grid, const CUtensorMap& gmap, int smem, const sp::SpArgs& a, int nblocks,
+// sparse-ligand engine k_corr_sparse<xts, zt, grid> (dock_sparse.cuh); xts = translations per lane along x
+cudaError_t dock_launch_sparse2(int zt, bool grid, const CUtensorMap& gmap, int smem, const sp::SpArgs& a, int nblocks,
                                 cudaStream_t st);
-cudaError_t dock_launch_sparse4(bool grid, const CUtensorMap& gmap, int smem, const sp::SpArgs& a, int nblocks,
+cudaError_t dock_launch_sparse4(int zt, bool grid, const CUtensorMap& gmap, int smem, const sp::SpArgs& a, int nblocks,
                                 cudaStream_t st);
-cudaError_t dock_launch_sparse5(bool grid, const CUtensorMap& gmap, int smem, const sp::SpArgs& a, int nblocks,
+cudaError_t dock_launch_sparse5(int zt, bool grid, const CUtensorMap& gmap, int smem, const sp::SpArgs& a, int nblocks,
                                 cudaStream_t st);
-inline cudaError_t dock_launch_sparse(int xts, bool grid, const CUtensorMap& gmap, int smem, const sp::SpArgs& a,
-                                      int nblocks, cudaStream_t st)
+inline cudaError_t dock_launch_sparse(int xts, int zt, bool grid, const CUtensorMap& gmap, int smem,
+                                      const sp::SpArgs& a, int nblocks, cudaStream_t st)
 {
     switch (xts) {
-        case 2: return dock_launch_sparse2(grid, gmap, smem, a, nblocks, st);
-        case 4: return dock_launch_sparse4(grid, gmap, smem, a, nblocks, st);
-        case 5: return dock_launch_sparse5(grid, gmap, smem, a, nblocks, st);
+        case 2: return dock_launch_sparse2(zt, grid, gmap, smem, a, nblocks, st);
+        case 4: return dock_launch_sparse4(zt, grid, gmap, smem, a, nblocks, st);
+        case 5: return dock_launch_sparse5(zt, grid, gmap, smem, a, nblocks, st);
         default: return cudaErrorInvalidValue;
     }
 }

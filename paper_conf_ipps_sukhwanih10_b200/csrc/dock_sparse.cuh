@@ -20,8 +20,9 @@
 //
 // k_corr_sparse: one CTA = (group of RB rotations of one probe, range of columns of TX x TY x nz translations).
 // The producer warp streams z-planes of every atom grid G_a (TMA, one box [TY+m-1][TX+m-1] per atom and
-// plane) through a ring of NPL plane slots; 8 consumer warps = TY rows x PZ planes per step; lane j owns
-// the translations x0 + j + 32 i (i < XTS), so every shared-memory read of a warp is 32 consecutive words
+// plane) through a ring of NPL plane slots; 8 consumer warps = TY rows x 2 plane groups of ZT planes per
+// step (ZT = 2 for 64-translation rows, else 1); lane j owns the translations x0 + j + 32 i (i < XTS) of
+// its row in each of its planes, so every shared-memory read of a warp is 32 consecutive words
 // (conflict-free for any voxel offset).  Per rotation the occupied voxels' terms are gathered from the
 // ring, then the per-warp top-32 key lists of the FFMA engine take the scores (no score grid in HBM);
 // item end publishes bound / mu / candidates for k_merge exactly like the other engines.
@@ -35,8 +36,10 @@ using dk::KEY_MAX;
 
 constexpr int RB = 8;                     // rotations per item (accumulated side by side: independent chains)
 constexpr int TY = 4;                     // translation rows per column
-constexpr int PZ = 2;                     // output planes per step
-constexpr int NWC = TY * PZ;              // consumer warps
+constexpr int NPG = 2;                    // plane groups per step (warps = TY rows x NPG groups)
+constexpr int NWC = TY * NPG;             // consumer warps
+// ZT = planes per warp and step (a template parameter): 2 for the narrow 64-translation rows when the plane
+// ring fits (more values per term decode and per gate), else 1; a step advances NPG * ZT planes
 constexpr int NTHREADS = (NWC + 1) * 32;  // + 1 TMA producer warp
 constexpr int TMAX = 32;                  // occupied voxels per rotation (= atoms) handled by the engine
 constexpr int NPLMAX = 16;                // plane-ring depth limit
@@ -240,15 +243,16 @@ struct Vec {   // passed by value to the out-of-line helpers (a pointer would fo
     float v[N];
 };
 
-template <int XTS>
-__device__ __noinline__ void sp_insert(unsigned long long* L, float2* th_rec, const Vec<XTS> acc, unsigned vmask,
-                                       uint32_t tbase, int lane)
+template <int XTS, int ZT>
+__device__ __noinline__ void sp_insert(unsigned long long* L, float2* th_rec, const Vec<XTS * ZT> acc, unsigned vmask,
+                                       uint32_t tbase, uint32_t plane_stride, int lane)
 {
     unsigned long long lst = L[lane];
     unsigned long long thk = dk::shfl_u64(lst, 31);
 #pragma unroll
-    for (int i = 0; i < XTS; i++) {
-        const unsigned long long key = ((vmask >> i) & 1u) ? dk::make_key(acc.v[i], tbase + 32 * i) : KEY_MAX;
+    for (int v = 0; v < XTS * ZT; v++) {
+        const uint32_t t = tbase + static_cast<uint32_t>(v / XTS) * plane_stride + 32u * static_cast<uint32_t>(v % XTS);
+        const unsigned long long key = ((vmask >> v) & 1u) ? dk::make_key(acc.v[v], t) : KEY_MAX;
         unsigned mm = __ballot_sync(FULL, key < thk);
         while (mm) {
             const int src = __ffs(mm) - 1;
@@ -289,9 +293,10 @@ __device__ __noinline__ Vec<XTS> sp_direct(const float* wv, int P, const float* 
     return d;
 }
 
-template <int XTS, bool GRID>
+template <int XTS, int ZT, bool GRID>
 __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_constant__ CUtensorMap gmap, const SpArgs a)
 {
+    constexpr int PZ = NPG * ZT, V = XTS * ZT;   // planes per step; values per lane and rotation
     extern __shared__ __align__(128) unsigned char smem[];
     __shared__ uint64_t full[NPLMAX], empty[NPLMAX];
     __shared__ int4 s_term[TMAX * RB];   // [term][rotation]: (byte offset (atom ring + (vy * TXB + vx) * 4),
@@ -380,8 +385,8 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
         return;
     }
 
-    // ---------------- consumers: warp = (row ry, plane pz of the step)
-    const int ry = warp % TY, pz = warp / TY;
+    // ---------------- consumers: warp = (row ry, plane group pg: planes pg * ZT .. pg * ZT + ZT - 1 of a step)
+    const int ry = warp % TY, pg = warp / TY;
     unsigned long long(*lists)[32] = s_lst[warp];
 #pragma unroll
     for (int r = 0; r < RB; r++) lists[r][lane] = KEY_MAX;
@@ -389,8 +394,9 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
     __syncwarp();
     const uint32_t lane_base = dk::smem_u32(ring) + 4u * static_cast<uint32_t>(ry * a.TXB + lane);
     const uint32_t ring_bytes = static_cast<uint32_t>(npl * slot_bytes);
+    const uint32_t plane_stride = static_cast<uint32_t>(a.nx * a.ny);
     int waited = 0, cbase = 0;
-    int pslot = pz;   // ring slot of this warp's plane (cbase + zabs) mod npl, maintained incrementally
+    int pslot = (pg * ZT) % npl;   // ring slot of this warp's first plane, maintained incrementally
     for (int c = c0; c < c1; c++, cbase += n_planes) {
         const int tx = c % a.ntx, ty = c / a.ntx;
         const int y = ty * TY + ry;
@@ -398,7 +404,6 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
         unsigned xmask = 0;
 #pragma unroll
         for (int i = 0; i < XTS; i++) xmask |= (xb + 32 * i < a.nx) ? (1u << i) : 0u;
-        const bool xfull = __all_sync(FULL, xmask == (1u << XTS) - 1u);   // no masked x (uniform)
         int zz = 0;
         for (; zz < a.nz; zz += PZ) {
             const int need = cbase + min(zz + PZ - 1 + M - 1, n_planes - 1);
@@ -406,45 +411,62 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
                 dk::mbar_wait(&full[waited % npl], (waited / npl) & 1);
                 waited++;
             }
-            const int zabs = zz + pz;
-            const uint32_t zoff = static_cast<uint32_t>(pslot * slot_bytes);
-            // a warp whose plane or row lies outside the grid skips the step (its ring slots may already hold
-            // later planes); the condition is warp-uniform
-            if (zabs < a.nz && y < a.ny) {
-                const unsigned vmask = xmask;
-                const uint32_t tbase = static_cast<uint32_t>((zabs * a.ny + y) * a.nx + xb);
+            const int z0w = zz + pg * ZT;   // this warp's first plane
+            // a warp whose first plane or row lies outside the grid skips the step (its ring slots may already
+            // hold later planes); the condition is warp-uniform.  A later plane beyond the grid reads the first
+            // plane's slot (masked out).
+            if (z0w < a.nz && y < a.ny) {
+                unsigned vmask = 0;
+                uint32_t zoff[ZT];
+#pragma unroll
+                for (int j = 0; j < ZT; j++) {
+                    const bool pj = z0w + j < a.nz;
+                    int sj = pslot + j;
+                    sj = sj >= npl ? sj - npl : sj;
+                    zoff[j] = static_cast<uint32_t>((pj ? sj : pslot) * slot_bytes);
+                    vmask |= pj ? (xmask << (j * XTS)) : 0u;
+                }
+                const bool vfull = __all_sync(FULL, vmask == (1u << V) - 1u);   // nothing masked (uniform)
+                const uint32_t tbase = static_cast<uint32_t>((z0w * a.ny + y) * a.nx + xb);
                 // term-outer, rotation-inner, branch-free: the RB rotations' gathers are independent (weight 1 for
                 // a single-atom voxel, 0 for an absent or multi-atom term: fma(1, g, acc) == acc + g exactly);
                 // term 0 initialises the accumulators
-                float acc[RB][XTS];
+                float acc[RB][V];
                 if (tmax > 0) {
 #pragma unroll
                     for (int r = 0; r < RB; r++) {
                         const int4 term = s_term[r];
-                        uint32_t zo = zoff + static_cast<uint32_t>(term.y);
-                        zo = zo >= ring_bytes ? zo - ring_bytes : zo;
-                        const uint32_t ad = lane_base + zo + static_cast<uint32_t>(term.x);
                         const float wt = __int_as_float(term.z);
 #pragma unroll
-                        for (int i = 0; i < XTS; i++) acc[r][i] = wt * lds_f32(ad + 128u * i);
+                        for (int j = 0; j < ZT; j++) {
+                            uint32_t zo = zoff[j] + static_cast<uint32_t>(term.y);
+                            zo = zo >= ring_bytes ? zo - ring_bytes : zo;
+                            const uint32_t ad = lane_base + zo + static_cast<uint32_t>(term.x);
+#pragma unroll
+                            for (int i = 0; i < XTS; i++) acc[r][j * XTS + i] = wt * lds_f32(ad + 128u * i);
+                        }
                     }
                 } else {   // a probe without atoms scores 0 everywhere
 #pragma unroll
                     for (int r = 0; r < RB; r++)
 #pragma unroll
-                        for (int i = 0; i < XTS; i++) acc[r][i] = 0.0f;
+                        for (int v = 0; v < V; v++) acc[r][v] = 0.0f;
                 }
 #pragma unroll 1
                 for (int t = 1; t < tmax; t++) {
 #pragma unroll
                     for (int r = 0; r < RB; r++) {
                         const int4 term = s_term[t * RB + r];
-                        uint32_t zo = zoff + static_cast<uint32_t>(term.y);
-                        zo = zo >= ring_bytes ? zo - ring_bytes : zo;
-                        const uint32_t ad = lane_base + zo + static_cast<uint32_t>(term.x);
                         const float wt = __int_as_float(term.z);
 #pragma unroll
-                        for (int i = 0; i < XTS; i++) acc[r][i] = fmaf(wt, lds_f32(ad + 128u * i), acc[r][i]);
+                        for (int j = 0; j < ZT; j++) {
+                            uint32_t zo = zoff[j] + static_cast<uint32_t>(term.y);
+                            zo = zo >= ring_bytes ? zo - ring_bytes : zo;
+                            const uint32_t ad = lane_base + zo + static_cast<uint32_t>(term.x);
+#pragma unroll
+                            for (int i = 0; i < XTS; i++)
+                                acc[r][j * XTS + i] = fmaf(wt, lds_f32(ad + 128u * i), acc[r][j * XTS + i]);
+                        }
                     }
                 }
                 if (has_direct) {
@@ -455,12 +477,15 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
                         for (int r = 0; r < RB; r++) {
                             const int code = s_dterm[t * RB + r];
                             if (code >= 0) {
-                                const Vec<XTS> d = sp_direct<XTS>(
-                                    a.dw + (static_cast<size_t>(gr.slot0 + r) * TMAX + (code >> 24)) * a.P, a.P, a.rec,
-                                    a.rXp, a.rYp, a.rZp, zabs + ((code >> 16) & 0xff), y + ((code >> 8) & 0xff),
-                                    xb + (code & 0xff), vmask);
 #pragma unroll
-                                for (int i = 0; i < XTS; i++) acc[r][i] += d.v[i];
+                                for (int j = 0; j < ZT; j++) {
+                                    const Vec<XTS> d = sp_direct<XTS>(
+                                        a.dw + (static_cast<size_t>(gr.slot0 + r) * TMAX + (code >> 24)) * a.P, a.P,
+                                        a.rec, a.rXp, a.rYp, a.rZp, z0w + j + ((code >> 16) & 0xff),
+                                        y + ((code >> 8) & 0xff), xb + (code & 0xff), (vmask >> (j * XTS)) & xmask);
+#pragma unroll
+                                    for (int i = 0; i < XTS; i++) acc[r][j * XTS + i] += d.v[i];
+                                }
                             }
                         }
                     }
@@ -471,26 +496,26 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
                         if (r < nrot) {
                             float* out = a.grid + static_cast<size_t>(grp + r) * a.nx * a.ny * a.nz + tbase;
 #pragma unroll
-                            for (int i = 0; i < XTS; i++)
-                                if ((vmask >> i) & 1u) out[32 * i] = acc[r][i];
+                            for (int v = 0; v < V; v++)
+                                if ((vmask >> v) & 1u) out[(v / XTS) * plane_stride + 32 * (v % XTS)] = acc[r][v];
                         }
                     }
                 } else {
                     // exact gate of every rotation at once: a strictly better score, or a tie whose t_lin could
-                    // precede the list's 32nd key; one warp vote for all RB rotations
+                    // precede the list's 32nd key (tbase is the smallest t_lin of the lane); one warp vote for all
                     unsigned pass = 0;
 #pragma unroll
                     for (int r = 0; r < RB; r++) {
                         const float2 thr = s_th[warp][r];
                         float mn;
-                        if (xfull) {
+                        if (vfull) {
                             mn = acc[r][0];
 #pragma unroll
-                            for (int i = 1; i < XTS; i++) mn = fminf(mn, acc[r][i]);
+                            for (int v = 1; v < V; v++) mn = fminf(mn, acc[r][v]);
                         } else {
                             mn = __int_as_float(0x7f800000);
 #pragma unroll
-                            for (int i = 0; i < XTS; i++) mn = ((vmask >> i) & 1u) ? fminf(mn, acc[r][i]) : mn;
+                            for (int v = 0; v < V; v++) mn = ((vmask >> v) & 1u) ? fminf(mn, acc[r][v]) : mn;
                         }
                         const bool any = mn < thr.x || (mn == thr.x && tbase < __float_as_uint(thr.y));
                         pass |= (any && r < nrot) ? (1u << r) : 0u;
@@ -500,10 +525,10 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
 #pragma unroll
                         for (int r = 0; r < RB; r++) {
                             if ((pass >> r) & 1u) {
-                                Vec<XTS> av;
+                                Vec<V> av;
 #pragma unroll
-                                for (int i = 0; i < XTS; i++) av.v[i] = acc[r][i];
-                                sp_insert<XTS>(lists[r], &s_th[warp][r], av, vmask, tbase, lane);
+                                for (int v = 0; v < V; v++) av.v[v] = acc[r][v];
+                                sp_insert<XTS, ZT>(lists[r], &s_th[warp][r], av, vmask, tbase, plane_stride, lane);
                             }
                         }
                     }
@@ -522,7 +547,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
         if (lane == 0)
             for (int j = zz; j < n_planes; j++) dk::mbar_arrive(&empty[(cbase + j) % npl]);
         __syncwarp();
-        pslot = (cbase + n_planes + pz) % npl;
+        pslot = (cbase + n_planes + pg * ZT) % npl;
     }
 
     if constexpr (!GRID) {
