@@ -395,7 +395,8 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
     const uint32_t lane_base = dk::smem_u32(ring) + 4u * static_cast<uint32_t>(ry * a.TXB + lane);
     const uint32_t ring_bytes = static_cast<uint32_t>(npl * slot_bytes);
     const uint32_t plane_stride = static_cast<uint32_t>(a.nx * a.ny);
-    int waited = 0, cbase = 0;
+    int waited = 0, cbase = 0, wslot = 0, rslot = 0;   // next plane to wait for (slot), next plane to release
+    unsigned wphase = 0;
     int pslot = (pg * ZT) % npl;   // ring slot of this warp's first plane, maintained incrementally
     for (int c = c0; c < c1; c++, cbase += n_planes) {
         const int tx = c % a.ntx, ty = c / a.ntx;
@@ -407,9 +408,13 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
         int zz = 0;
         for (; zz < a.nz; zz += PZ) {
             const int need = cbase + min(zz + PZ - 1 + M - 1, n_planes - 1);
-            while (waited <= need) {
-                dk::mbar_wait(&full[waited % npl], (waited / npl) & 1);
+            while (waited <= need) {   // ring slot / phase of plane `waited` tracked without divisions
+                dk::mbar_wait(&full[wslot], wphase);
                 waited++;
+                if (++wslot == npl) {
+                    wslot = 0;
+                    wphase ^= 1u;
+                }
             }
             const int z0w = zz + pg * ZT;   // this warp's first plane
             // a warp whose first plane or row lies outside the grid skips the step (its ring slots may already
@@ -535,19 +540,24 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
                 }
             }
             __syncwarp();
-            if (lane == 0) {
 #pragma unroll
-                for (int q = 0; q < PZ; q++)
-                    if (zz + q < n_planes) dk::mbar_arrive(&empty[(cbase + zz + q) % npl]);
+            for (int q = 0; q < PZ; q++) {
+                if (zz + q < n_planes) {
+                    if (lane == 0) dk::mbar_arrive(&empty[rslot]);
+                    rslot = rslot + 1 == npl ? 0 : rslot + 1;
+                }
             }
             pslot += PZ;
             pslot = pslot >= npl ? pslot - npl : pslot;
         }
         // column end: release its remaining halo planes; the next column's planes follow in the ring
-        if (lane == 0)
-            for (int j = zz; j < n_planes; j++) dk::mbar_arrive(&empty[(cbase + j) % npl]);
+        for (int j = zz; j < n_planes; j++) {
+            if (lane == 0) dk::mbar_arrive(&empty[rslot]);
+            rslot = rslot + 1 == npl ? 0 : rslot + 1;
+        }
         __syncwarp();
-        pslot = (cbase + n_planes + pg * ZT) % npl;
+        pslot = rslot + pg * ZT;   // the next column's first plane is the next one to be released
+        pslot = pslot >= npl ? pslot - npl : pslot;
     }
 
     if constexpr (!GRID) {
