@@ -808,15 +808,21 @@ dock_status sp_prepare(dock_ctx* ctx, int m, const dock_probe_desc* probes, int 
     return DOCK_OK;
 }
 
-// Cost model of the engine choice (auto): gathered values per SM-clock of the sparse engine vs executed
-// bf16 MACs per SM-clock of the tensor-core engine (bf16x3 with the PAIR scheme: 3 per algorithmic MAC),
-// both measured on B200: ~6 gathers and ~3000 MACs per clock and SM.
-bool sp_better(const dock_ctx* ctx, const SpCall& sc, int m, int n_units)
+// Cost model of the engine choice (auto), per SM-clock rates measured on B200: the sparse
+// engine gathers ~6 values (one per occupied voxel and translation); the tensor-core engine executes ~3000
+// bf16 MACs (K-steps of 16 per rotation and translation, its bf16x3 split and padding included); the FFMA
+// engine ~170 FP32 FMAs.
+bool sp_better(dock_ctx* ctx, const SpCall& sc, int m, int n_units)
 {
     if (!sc.ok) return false;
     const double ncell = (double)ctx->nx * ctx->ny * ctx->nz;
     const double sparse = sc.terms * ncell / 6.0;
-    const double dense = double(n_units) * ncell * ctx->P * m * m * m * 3.0 / 3000.0;
+    int v = 0, G = 0;
+    double dense;
+    if (plan_tc_launch(ctx, m, tc::ROT, &v, &G))
+        dense = double(n_units) * ncell * ctx->tcplan[v][m].nsteps * 16.0 / 3000.0;
+    else
+        dense = double(n_units) * ncell * ctx->P * m * m * m / 170.0;
     return sparse < dense;
 }
 

@@ -269,6 +269,31 @@ __device__ __noinline__ void sp_insert(unsigned long long* L, float2* th_rec, co
     __syncwarp();
 }
 
+// mbarrier wait on a 32-bit shared address (no generic-to-shared conversion in the loop)
+__device__ __forceinline__ void mbar_wait_s(uint32_t bar, unsigned parity)
+{
+    uint32_t ok;
+    asm volatile(
+        "{\n\t.reg .pred p;\n\tmbarrier.try_wait.parity.shared::cta.b64 p, [%1], %2;\n\tselp.u32 %0, 1, 0, p;\n}\n"
+        : "=r"(ok)
+        : "r"(bar), "r"(parity)
+        : "memory");
+    if (ok) return;
+    const long long t0 = clock64();
+    do {
+        asm volatile(
+            "{\n\t.reg .pred p;\n\tmbarrier.try_wait.parity.shared::cta.b64 p, [%1], %2;\n\tselp.u32 %0, 1, 0, p;\n}\n"
+            : "=r"(ok)
+            : "r"(bar), "r"(parity)
+            : "memory");
+        if (clock64() - t0 > (1ll << 35)) __trap();
+    } while (!ok);
+}
+__device__ __forceinline__ void mbar_arrive_s(uint32_t bar)
+{
+    asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(bar) : "memory");
+}
+
 __device__ __forceinline__ float lds_f32(uint32_t addr)
 {
     float v;
@@ -395,6 +420,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
     const uint32_t lane_base = dk::smem_u32(ring) + 4u * static_cast<uint32_t>(ry * a.TXB + lane);
     const uint32_t ring_bytes = static_cast<uint32_t>(npl * slot_bytes);
     const uint32_t plane_stride = static_cast<uint32_t>(a.nx * a.ny);
+    const uint32_t full_s = dk::smem_u32(full), empty_s = dk::smem_u32(empty);
     int waited = 0, cbase = 0, wslot = 0, rslot = 0;   // next plane to wait for (slot), next plane to release
     unsigned wphase = 0;
     int pslot = (pg * ZT) % npl;   // ring slot of this warp's first plane, maintained incrementally
@@ -409,7 +435,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
         for (; zz < a.nz; zz += PZ) {
             const int need = cbase + min(zz + PZ - 1 + M - 1, n_planes - 1);
             while (waited <= need) {   // ring slot / phase of plane `waited` tracked without divisions
-                dk::mbar_wait(&full[wslot], wphase);
+                mbar_wait_s(full_s + 8u * wslot, wphase);
                 waited++;
                 if (++wslot == npl) {
                     wslot = 0;
@@ -543,7 +569,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
 #pragma unroll
             for (int q = 0; q < PZ; q++) {
                 if (zz + q < n_planes) {
-                    if (lane == 0) dk::mbar_arrive(&empty[rslot]);
+                    if (lane == 0) mbar_arrive_s(empty_s + 8u * rslot);
                     rslot = rslot + 1 == npl ? 0 : rslot + 1;
                 }
             }
@@ -552,7 +578,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
         }
         // column end: release its remaining halo planes; the next column's planes follow in the ring
         for (int j = zz; j < n_planes; j++) {
-            if (lane == 0) dk::mbar_arrive(&empty[rslot]);
+            if (lane == 0) mbar_arrive_s(empty_s + 8u * rslot);
             rslot = rslot + 1 == npl ? 0 : rslot + 1;
         }
         __syncwarp();
