@@ -92,9 +92,8 @@ struct dock_ctx {
     TcPlan tcplan[3][DOCK_MAX_M + 1];   // [variant][m]
     DevBuf Wtc;
     // diagnostics (environment, read at init): DOCK_TC_TRACE=1 prints per-role cycle counters of every
-    // k_corr_tc launch to stderr; DOCK_TC_DEBUG=1|2 disables parts of the epilogue (timing only)
+    // tcgen05 launch to stderr
     unsigned long long* d_trace = nullptr;
-    int tc_dbg = 0;
     // per-call scratch (grow-only)
     DevBuf xyz, coef, off, rot, Lw, T, mu, cnt, cand, poses, fb_list, grid, slots, units, Lw_fb, picks;
     int* d_small = nullptr;    // [0] status bits (sticky until the next sync point), [1] fb_cnt, [2] cand_max
@@ -659,7 +658,6 @@ tc::TcArgs tc_args(dock_ctx* ctx, int m, int v, int n_slots, int G, const unsign
     a.wstages = tp.wstages;
     a.nepi = ctx->tc_nepi > 0 ? std::min(tc::NEPI_MAX, ctx->tc_nepi) : tc::NEPI_MAX;
     a.trace = ctx->d_trace;
-    a.dbg = ctx->tc_dbg;
     return a;
 }
 
@@ -1411,7 +1409,6 @@ dock_status dock_init(const dock_grid_desc* g, const float* receptor, const floa
         return bail(DOCK_E_CUDA);
     for (auto& st : ctx->stage)
         if (cudaEventCreateWithFlags(&st.ev, cudaEventDisableTiming) != cudaSuccess) return bail(DOCK_E_CUDA);
-    if (const char* e = getenv("DOCK_TC_DEBUG")) ctx->tc_dbg = atoi(e);
     if (const char* e = getenv("DOCK_TC_TRACE")) {
         if (atoi(e) > 0 && cudaMalloc(&ctx->d_trace, sizeof(unsigned long long) * tc::TR_N) != cudaSuccess)
             return bail(DOCK_E_OOM);
@@ -1764,12 +1761,12 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
             const double c = h[tc::TR_CTAS] ? double(h[tc::TR_CTAS]) : 1.0;
             const double e = h[tc::TR_EPI_WARPS] ? double(h[tc::TR_EPI_WARPS]) : 1.0;
             fprintf(stderr,
-                    "TCTRACE {\"variant\": %d, \"dbg\": %d, \"ctas\": %llu, \"tiles_per_cta\": %.1f, "
+                    "TCTRACE {\"variant\": %d, \"ctas\": %llu, \"tiles_per_cta\": %.1f, "
                     "\"mma_total\": %.0f, \"mma_wait_tmem_empty\": %.0f, \"mma_wait_w_full\": %.0f, "
                     "\"mma_wait_rec_full\": %.0f, \"epi_total\": %.0f, \"epi_wait_tm_full\": %.0f, "
                     "\"epi_ldtm\": %.0f, \"prod_total\": %.0f, \"prod_wait_w_empty\": %.0f, "
                     "\"prod_wait_rec_empty\": %.0f}\n",
-                    v, ctx->tc_dbg, h[tc::TR_CTAS], h[tc::TR_TILES] / c, h[tc::TR_MMA_TOTAL] / c,
+                    v, h[tc::TR_CTAS], h[tc::TR_TILES] / c, h[tc::TR_MMA_TOTAL] / c,
                     h[tc::TR_MMA_TMEMPTY] / c, h[tc::TR_MMA_WFULL] / c, h[tc::TR_MMA_RFULL] / c,
                     h[tc::TR_EPI_TOTAL] / e, h[tc::TR_EPI_TMFULL] / e, h[tc::TR_EPI_LDTM] / e,
                     h[tc::TR_PROD_TOTAL] / c, h[tc::TR_PROD_WEMPTY] / c, h[tc::TR_PROD_REMPTY] / c);

@@ -70,11 +70,9 @@ struct TcArgs {
     // grid mode
     float* grid;
     const unsigned* n_live;     // optional (device): rotations >= *n_live are dead (device-driven fallback)
-    // diagnostics (DOCK_TC_TRACE / DOCK_TC_DEBUG environment variables; off on the product path):
-    // trace = per-role cycle counters summed over CTAs (see TR_*); dbg 1 = epilogue skips the TMEM
-    // drain, 2 = drain without candidate processing (timing experiments only: poses are invalid)
+    // diagnostics (DOCK_TC_TRACE environment variable; off on the product path):
+    // trace = per-role cycle counters summed over CTAs (see TR_*)
     unsigned long long* trace;
-    int dbg;
 };
 
 // trace counters (cycles summed over CTAs)
@@ -302,7 +300,7 @@ __device__ __forceinline__ void epi_tile(const TcArgs& a, uint32_t tmem, uint64_
         const int y = ty * Q + q, z = tz;
         const bool row_ok = rot_ok && y < a.ny && z < a.nz;
         const uint32_t tbase = static_cast<uint32_t>((z * a.ny + y) * a.nx + x0);
-        if (a.dbg == 1 || cls >= NCH) {   // diagnostic (no TMEM drain), or no chunk of this row for this class
+        if (cls >= NCH) {   // no chunk of this row for this class
             __syncwarp();
             if (lane == 0) dk::mbar_arrive(&tm_empty[q]);
             continue;
@@ -321,7 +319,7 @@ __device__ __forceinline__ void epi_tile(const TcArgs& a, uint32_t tmem, uint64_
             tc_fence_before();
             __syncwarp();
             if (lane == 0) dk::mbar_arrive(&tm_empty[q]);
-            if (!row_ok || a.dbg == 2) continue;
+            if (!row_ok) continue;
             float* grow = GRID ? a.grid + static_cast<size_t>(slot) * a.nx * a.ny * a.nz + tbase : nullptr;
             epi_chunk<GRID>(v0, lst, th, th_t, tbase, c0, min(32, a.nx - x0 - c0), grow);
             epi_chunk<GRID>(v1, lst, th, th_t, tbase, c1, min(32, a.nx - x0 - c1), grow);
@@ -339,7 +337,7 @@ __device__ __forceinline__ void epi_tile(const TcArgs& a, uint32_t tmem, uint64_
                 __syncwarp();
                 if (lane == 0) dk::mbar_arrive(&tm_empty[q]);
             }
-            if (!row_ok || a.dbg == 2) continue;
+            if (!row_ok) continue;
             epi_chunk<GRID>(v, lst, th, th_t, tbase, c0, min(32, a.nx - x0 - c0),
                             GRID ? a.grid + static_cast<size_t>(slot) * a.nx * a.ny * a.nz + tbase : nullptr);
         }
