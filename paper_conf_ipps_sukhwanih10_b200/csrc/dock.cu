@@ -116,6 +116,7 @@ struct dock_ctx {
     cudaStream_t cap_stream = nullptr, cap_stream2 = nullptr;   // private capture streams
     cudaGraphExec_t fb_exec = nullptr;
     unsigned char fb_key[256] = {0};
+    int fb_host_loop = 0;   // DOCK_FB_HOST_LOOP=1 (environment): fallback from a host loop instead of the graph
     DevBuf fb_grid, fb_Lw, fb_W, fb_picks, fb_slots, fb_ctl, fb_groups;
     // sparse-ligand engine: plans, atom grids G_a of the call, occupied-voxel term tables
     SpPlan spplan[DOCK_MAX_M + 1][6];   // [m][xts]
@@ -1078,19 +1079,93 @@ dock_status fb_buffers(dock_ctx* ctx, int m, int ch, int k)
 
 // Capture + instantiate the fallback graph for this key (ctx->stream is redirected to the private capture
 // streams while the existing launch helpers record into the graph).
+// One iteration of the fallback loop on stream st (the kernels read the chunk from the device-side control
+// block): chunk -> [voxelize] -> GRID correlation -> greedy rounds -> emit.  Captured into the WHILE body of
+// the fallback graph, or launched from a host loop (DOCK_FB_HOST_LOOP=1: sanitizer runs, whose tools do not
+// support conditional graph nodes).
+dock_status enqueue_fb_body(dock_ctx* ctx, const FbKey& key, const dk::FbDyn* d_dyn, const SpCall* sc, cudaStream_t st)
+{
+    const int m = key.m, ch = key.ch, k = key.k;
+    auto* fb_cnt = reinterpret_cast<unsigned int*>(ctx->d_small + 1);
+    auto* ctl = static_cast<dk::FbCtl*>(ctx->fb_ctl.p);
+    int* slots = static_cast<int*>(ctx->fb_slots.p);
+    cudaStream_t user = ctx->stream;
+    ctx->stream = st;   // the launch helpers below enqueue on ctx->stream
+    auto body = [&]() -> dock_status {
+        dk::k_fb_chunk<<<1, 128, 0, st>>>(fb_cnt, static_cast<const int*>(ctx->fb_list.p), ctl, slots, ch);
+        CU(cudaGetLastError());
+        const float* Lw = static_cast<const float*>(ctx->fb_Lw.p);
+        float* grid = static_cast<float*>(ctx->fb_grid.p);
+        if (key.kind == ENG_SPARSE) {
+            // the main pass's atom grids and term tables stay valid until the next call: one single-rotation
+            // group per flagged slot, GRID epilogue into row = chunk position
+            auto* groups = static_cast<sp::Group*>(ctx->fb_groups.p);
+            sp::k_sparse_fb_groups<<<(ch + 127) / 128, 128, 0, st>>>(
+                slots, &ctl->n_live, static_cast<const int*>(ctx->sp_slot_atoms.p), groups, ch);
+            CU(cudaGetLastError());
+            sp::SpArgs a = sp_args(ctx, *sc, groups, ch);
+            a.grid = grid;
+            a.n_live = &ctl->n_live;
+            CU(dock_launch_sparse(sc->xts, sc->zt, true, ctx->sp_tmap, sc->smem, a, (int)(ch * a.G), st));
+        } else {
+            const int nvox = (ch + dk::RB - 1) / dk::RB * dk::RB * ctx->P;
+            dk::k_voxelize_dyn<<<(nvox + 127) / 128, 128, 0, st>>>(&d_dyn->vox);
+            CU(cudaGetLastError());
+            if (key.kind == ENG_TC) {
+                TRY(pack_weights_tc(ctx, m, key.v, ch, Lw, &ctx->fb_W));
+                tc::TcArgs a = tc_args(ctx, m, key.v, ch, key.G, static_cast<const unsigned char*>(ctx->fb_W.p));
+                a.grid = grid;
+                a.n_live = &ctl->n_live;
+                a.trace = nullptr;
+                CU(launch_tc(m, key.v, true, ctx->tcplan[key.v][m], a, key.G, st));
+            } else {
+                const int64_t nb = (ch + dk::RB - 1) / dk::RB;
+                dk::CorrArgs a = corr_args(ctx, m, ch, key.G, Lw);
+                a.grid = grid;
+                a.n_live = &ctl->n_live;
+                CU(dock_launch_ffma(m, true, ctx->plan[m].tmap, ctx->plan[m].smem, a, (int)(nb * key.G), st));
+            }
+        }
+        dk::GreedyArgs ga{};
+        ga.grid = grid;
+        ga.slots = slots;
+        ga.picks = static_cast<unsigned long long*>(ctx->fb_picks.p);
+        ga.n = ch;
+        ga.k = k;
+        ga.rho = key.rho;
+        ga.nx = ctx->nx;
+        ga.ny = ctx->ny;
+        ga.nz = ctx->nz;
+        ga.flag_bits = 1u;   // DOCK_POSE_FALLBACK
+        ga.n_live = &ctl->n_live;
+        ga.dyn = d_dyn;
+        dk::k_fill_u64<<<1, 256, 0, st>>>(ga.picks, (size_t)ch * k, dk::KEY_MAX);
+        CU(cudaGetLastError());
+        const int per_grid = std::max(8, std::min(512, 16 * ctx->n_sms / std::max(1, ch)));
+        for (int j = 0; j < k; j++) {
+            ga.round = j;
+            dk::k_greedy_round<<<ch * per_grid, 256, 0, st>>>(ga);
+            CU(cudaGetLastError());
+        }
+        dk::k_greedy_emit<<<(ch * k + 127) / 128, 128, 0, st>>>(ga);
+        CU(cudaGetLastError());
+        return DOCK_OK;
+    };
+    const dock_status r = body();
+    ctx->stream = user;
+    return r;
+}
+
 dock_status build_fb_graph(dock_ctx* ctx, const FbKey& key, const dk::FbDyn* d_dyn, const SpCall* sc)
 {
     if (ctx->fb_exec) {
         cudaGraphExecDestroy(ctx->fb_exec);
         ctx->fb_exec = nullptr;
     }
-    const int m = key.m, ch = key.ch, k = key.k;
     auto* fb_cnt = reinterpret_cast<unsigned int*>(ctx->d_small + 1);
     auto* ctl = static_cast<dk::FbCtl*>(ctx->fb_ctl.p);
-    int* slots = static_cast<int*>(ctx->fb_slots.p);
-    cudaStream_t user = ctx->stream, cs = ctx->cap_stream, cs2 = ctx->cap_stream2;
+    cudaStream_t cs = ctx->cap_stream, cs2 = ctx->cap_stream2;
     cudaGraph_t graph = nullptr;
-    dock_status st = DOCK_OK;
     auto body = [&]() -> dock_status {
         CU(cudaStreamBeginCapture(cs, cudaStreamCaptureModeThreadLocal));
         cudaStreamCaptureStatus cst;
@@ -1114,74 +1189,15 @@ dock_status build_fb_graph(dock_ctx* ctx, const FbKey& key, const dk::FbDyn* d_d
         CU(cudaStreamUpdateCaptureDependencies(cs, &node, 1, cudaStreamSetCaptureDependencies));
         // loop body, captured on the second private stream
         CU(cudaStreamBeginCaptureToGraph(cs2, loop, nullptr, nullptr, 0, cudaStreamCaptureModeThreadLocal));
-        ctx->stream = cs2;
-        dk::k_fb_chunk<<<1, 128, 0, cs2>>>(fb_cnt, static_cast<const int*>(ctx->fb_list.p), ctl, slots, ch);
+        TRY(enqueue_fb_body(ctx, key, d_dyn, sc, cs2));
+        dk::k_fb_advance<<<1, 1, 0, cs2>>>(h, fb_cnt, ctl, key.ch);
         CU(cudaGetLastError());
-        const float* Lw = static_cast<const float*>(ctx->fb_Lw.p);
-        float* grid = static_cast<float*>(ctx->fb_grid.p);
-        if (key.kind != ENG_SPARSE) {
-            const int nvox = (ch + dk::RB - 1) / dk::RB * dk::RB * ctx->P;
-            dk::k_voxelize_dyn<<<(nvox + 127) / 128, 128, 0, cs2>>>(&d_dyn->vox);
-            CU(cudaGetLastError());
-        }
-        if (key.kind == ENG_SPARSE) {
-            // the main pass's atom grids and term tables stay valid until the next call: one single-rotation
-            // group per flagged slot, GRID epilogue into row = chunk position
-            auto* groups = static_cast<sp::Group*>(ctx->fb_groups.p);
-            sp::k_sparse_fb_groups<<<(ch + 127) / 128, 128, 0, cs2>>>(
-                slots, &ctl->n_live, static_cast<const int*>(ctx->sp_slot_atoms.p), groups, ch);
-            CU(cudaGetLastError());
-            sp::SpArgs a = sp_args(ctx, *sc, groups, ch);
-            a.grid = grid;
-            a.n_live = &ctl->n_live;
-            CU(dock_launch_sparse(sc->xts, sc->zt, true, ctx->sp_tmap, sc->smem, a, (int)(ch * a.G), cs2));
-        } else if (key.kind == ENG_TC) {
-            TRY(pack_weights_tc(ctx, m, key.v, ch, Lw, &ctx->fb_W));
-            tc::TcArgs a = tc_args(ctx, m, key.v, ch, key.G, static_cast<const unsigned char*>(ctx->fb_W.p));
-            a.grid = grid;
-            a.n_live = &ctl->n_live;
-            a.trace = nullptr;
-            CU(launch_tc(m, key.v, true, ctx->tcplan[key.v][m], a, key.G, cs2));
-        } else {
-            const int64_t nb = (ch + dk::RB - 1) / dk::RB;
-            dk::CorrArgs a = corr_args(ctx, m, ch, key.G, Lw);
-            a.grid = grid;
-            a.n_live = &ctl->n_live;
-            CU(dock_launch_ffma(m, true, ctx->plan[m].tmap, ctx->plan[m].smem, a, (int)(nb * key.G), cs2));
-        }
-        dk::GreedyArgs ga{};
-        ga.grid = grid;
-        ga.slots = slots;
-        ga.picks = static_cast<unsigned long long*>(ctx->fb_picks.p);
-        ga.n = ch;
-        ga.k = k;
-        ga.rho = key.rho;
-        ga.nx = ctx->nx;
-        ga.ny = ctx->ny;
-        ga.nz = ctx->nz;
-        ga.flag_bits = 1u;   // DOCK_POSE_FALLBACK
-        ga.n_live = &ctl->n_live;
-        ga.dyn = d_dyn;
-        dk::k_fill_u64<<<1, 256, 0, cs2>>>(ga.picks, (size_t)ch * k, dk::KEY_MAX);
-        CU(cudaGetLastError());
-        const int per_grid = std::max(8, std::min(512, 16 * ctx->n_sms / std::max(1, ch)));
-        for (int j = 0; j < k; j++) {
-            ga.round = j;
-            dk::k_greedy_round<<<ch * per_grid, 256, 0, cs2>>>(ga);
-            CU(cudaGetLastError());
-        }
-        dk::k_greedy_emit<<<(ch * k + 127) / 128, 128, 0, cs2>>>(ga);
-        CU(cudaGetLastError());
-        dk::k_fb_advance<<<1, 1, 0, cs2>>>(h, fb_cnt, ctl, ch);
-        CU(cudaGetLastError());
-        ctx->stream = user;
         CU(cudaStreamEndCapture(cs2, nullptr));
         CU(cudaStreamEndCapture(cs, &graph));
         CU(cudaGraphInstantiate(&ctx->fb_exec, graph, 0));
         return DOCK_OK;
     };
-    st = body();
-    ctx->stream = user;
+    const dock_status st = body();
     if (st != DOCK_OK) {   // leave no capture open on the private streams
         cudaGraph_t junk = nullptr;
         cudaStreamCaptureStatus cst;
@@ -1247,6 +1263,20 @@ dock_status launch_fallback(dock_ctx* ctx, int m, int kind, int k, int rho, cons
     key.slots = ctx->fb_slots.p;
     key.ctl = ctx->fb_ctl.p;
     key.w = ctx->d_w;
+    if (ctx->fb_host_loop) {   // diagnostic mode: the same kernels from a host loop (synchronises)
+        auto* ctl = static_cast<dk::FbCtl*>(ctx->fb_ctl.p);
+        CU(cudaMemcpyAsync(ctx->h_small, ctx->d_small, 16, cudaMemcpyDeviceToHost, ctx->stream));
+        CU(cudaStreamSynchronize(ctx->stream));
+        const int n = ctx->h_small[1];
+        dk::k_fb_init_plain<<<1, 1, 0, ctx->stream>>>(ctl);
+        CU(cudaGetLastError());
+        for (int done = 0; done < n; done += ch) {
+            TRY(enqueue_fb_body(ctx, key, d_dyn, sc, ctx->stream));
+            dk::k_fb_advance_plain<<<1, 1, 0, ctx->stream>>>(ctl, ch);
+            CU(cudaGetLastError());
+        }
+        return DOCK_OK;
+    }
     if (!ctx->fb_exec || memcmp(&key, ctx->fb_key, sizeof(key)) != 0) {
         TRY(build_fb_graph(ctx, key, d_dyn, sc));
         memcpy(ctx->fb_key, &key, sizeof(key));
@@ -1409,6 +1439,7 @@ dock_status dock_init(const dock_grid_desc* g, const float* receptor, const floa
         return bail(DOCK_E_CUDA);
     for (auto& st : ctx->stage)
         if (cudaEventCreateWithFlags(&st.ev, cudaEventDisableTiming) != cudaSuccess) return bail(DOCK_E_CUDA);
+    if (const char* e = getenv("DOCK_FB_HOST_LOOP")) ctx->fb_host_loop = atoi(e);
     if (const char* e = getenv("DOCK_TC_TRACE")) {
         if (atoi(e) > 0 && cudaMalloc(&ctx->d_trace, sizeof(unsigned long long) * tc::TR_N) != cudaSuccess)
             return bail(DOCK_E_OOM);

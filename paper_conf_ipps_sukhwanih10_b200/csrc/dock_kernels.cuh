@@ -769,6 +769,13 @@ __global__ void k_fb_chunk(const unsigned int* fb_cnt, const int* fb_list, FbCtl
     for (int i = threadIdx.x; i < ch; i += blockDim.x) slots[i] = i < static_cast<int>(n) ? fb_list[pos + i] : 0;
     if (threadIdx.x == 0) ctl->n_live = n;
 }
+// host-loop variants (diagnostic mode, no conditional handle)
+__global__ void k_fb_init_plain(FbCtl* ctl)
+{
+    ctl->pos = 0;
+    ctl->n_live = 0;
+}
+__global__ void k_fb_advance_plain(FbCtl* ctl, int ch) { ctl->pos += static_cast<unsigned>(ch); }
 __global__ void k_fb_advance(cudaGraphConditionalHandle h, const unsigned int* fb_cnt, FbCtl* ctl, int ch)
 {
     const unsigned pos = ctl->pos + static_cast<unsigned>(ch);
