@@ -570,3 +570,40 @@ def test_empty_unit_range(D):
     out = D.dock_probe_batch(ctx, g.probes(1, m, P), g.rotations(4), unit_begin=2, unit_end=2, k=4, rho=1)
     assert len(out) == 0
     ctx.close()
+
+
+def test_sparse_engine_edge_cases(D, orc):
+    """Sparse-ligand engine limits: a probe without atoms scores 0 everywhere (exact ties -> the greedy picks
+    t_lin 0, 2, 4, 6 at rho = 1, tests/golden/filter_constant_grid.txt's reading); a 20-atom probe (about the
+    most whose plane ring fits shared memory at m = 4 on 64-translation rows; many multi-atom voxels -> direct
+    terms) matches the oracle; 33 atoms (> sp::TMAX) is refused when forced and routed to a dense engine by
+    auto."""
+    P, m = 3, 4
+    R = g.receptor_ftmap_like((40, 24, 20), P)
+    w = g.weights(P)
+    rot = g.rotations(5)
+    ctx = _ctx(D, R, w, m, 4)
+    empty = g.Probe(np.zeros((0, 3)), np.zeros((0, P), np.float32), m)
+    poses = D.dock_probe_batch(ctx, [empty], rot, k=4, rho=1)
+    assert (poses["score"] == 0).all() and (poses["t_lin"] == np.array([0, 2, 4, 6])).all()
+    rng = np.random.default_rng(32)
+    xyz = rng.normal(size=(20, 3))
+    xyz *= (1.5 * rng.random(20) ** (1 / 3) / np.linalg.norm(xyz, axis=1))[:, None]   # inside the box under rotation
+    big = g.Probe(xyz, rng.normal(size=(20, P)).astype(np.float32), m)
+    poses = D.dock_probe_batch(ctx, [big], rot, k=4, rho=1)
+    assert D.dock_get_info(ctx)["engine_last"] == 4
+    for r in range(len(rot)):
+        L = orc.voxelize(big.xyz, big.coef, m, rot[r], H)
+        S, A = orc.score_grid(R, L, w)
+        validate_unit(S, A, poses[r]["t_lin"], poses[r]["score"], 4, 1)
+    S_g = D.dock_score_grid(ctx, big, rot[2])
+    S_o, A_o = _oracle_SA(orc, R, w, big, rot[2])
+    assert (np.abs(S_g.astype(np.float64) - S_o) <= 1e-4 * A_o + 1e-12).all()
+    huge = g.Probe(np.zeros((33, 3)), np.ones((33, P), np.float32), m)
+    with pytest.raises(D.DockError) as e:
+        D.dock_probe_batch(ctx, [huge], rot, k=4, rho=1)
+    assert e.value.status == -2
+    D.dock_set_tuning(ctx, D.DOCK_TUNE_ENGINE, 0)
+    D.dock_probe_batch(ctx, [huge], rot, k=4, rho=1)
+    assert D.dock_get_info(ctx)["engine_last"] in (1, 2)
+    ctx.close()
