@@ -5,10 +5,12 @@
 //   k_em_self   (a)  per (conformation, atom): s_a over its forward + reverse pair segments -> Born radius
 //   k_em_pair   (b)  per (conformation, pair): GB + vdW energies, dE/dr at fixed radii, dE/dalpha_i,j
 //   k_em_chain       per (conformation, atom): c_a = dE/ds_a (self energy + GB through the Born radius)
-//   k_em_force  (c)  per (conformation, atom): F_a from its segments (pair terms + chain-rule terms)
+//   k_em_force  (c)  per (conformation, atom): F_a from its segments (pair terms + chain-rule terms; the
+//                    self-term derivatives of both sides come from k_em_self, which evaluates each once)
 //   k_em_energy      per conformation: the three totals (fixed-order block reduction)
 // The split forward/reverse pairs lists of P:L799-881 are the two segment tables built at init; every
-// accumulation is one thread walking its segments in pair order: deterministic, no atomics.  FP64.
+// per-atom accumulation is one warp over the atom's segments (lane-strided, then a fixed xor tree):
+// deterministic, no atomics.  FP64.
 #include <cuda_runtime.h>
 
 #include <algorithm>
@@ -62,28 +64,52 @@ __device__ __forceinline__ double dist(const double* xc, int a, int b, double& d
     return sqrt(dx * dx + dy * dy + dz * dz);
 }
 
+// One warp per (conformation, atom): lane l takes the atom's neighbours l, l + 32, ... of its forward then
+// reverse segment, and the lane partial sums are combined by a fixed xor tree -- deterministic, independent of
+// the batch, 32 gathers in flight per atom.
+__device__ __forceinline__ double warp_sum(double v)
+{
+#pragma unroll
+    for (int o = 16; o > 0; o >>= 1) v += __shfl_xor_sync(0xffffffffu, v, o);
+    return v;
+}
+// neighbour j of atom a (forward segment first): pair index and partner atom
+__device__ __forceinline__ void neighbour(const Sys& S, int a, int nf, int j, int& p, int& k)
+{
+    if (j < nf) {
+        p = S.fwd_off[a] + j;
+        k = S.pairs[p].y;
+    } else {
+        p = S.rev_pair[S.rev_off[a] + j - nf];
+        k = S.pairs[p].x;
+    }
+}
+
 // (a) self energies: s_a = 1/(2 eps_s R_a) + sum over a's neighbours (Eq. 5), Born radius (reading E3)
 __global__ void k_em_self(Sys S, const double* __restrict__ x, int nconf, double* s_out, double* alpha_out,
-                          double* eself)
+                          double* eself, double2* dsd)
 {
-    const long long idx = blockIdx.x * static_cast<long long>(blockDim.x) + threadIdx.x;
-    if (idx >= static_cast<long long>(nconf) * S.n) return;
-    const int c = static_cast<int>(idx / S.n), a = static_cast<int>(idx % S.n);
+    const long long w = (blockIdx.x * static_cast<long long>(blockDim.x) + threadIdx.x) >> 5;
+    const int lane = threadIdx.x & 31;
+    if (w >= static_cast<long long>(nconf) * S.n) return;   // warp-uniform
+    const int c = static_cast<int>(w / S.n), a = static_cast<int>(w % S.n);
     const double* xc = x + static_cast<size_t>(c) * S.n * 3;
-    double s = 1.0 / (2.0 * S.eps_s * S.R[a]), dx, dy, dz, t, dt;
-    for (int p = S.fwd_off[a]; p < S.fwd_off[a + 1]; p++) {
-        const int k = S.pairs[p].y;
+    const int nf = S.fwd_off[a + 1] - S.fwd_off[a], nn = nf + S.rev_off[a + 1] - S.rev_off[a];
+    double s = 0.0, dx, dy, dz, t, dt;
+    double* ds_out = reinterpret_cast<double*>(dsd + static_cast<size_t>(c) * S.np);
+    for (int j = lane; j < nn; j += 32) {
+        int p, k;
+        neighbour(S, a, nf, j, p, k);
         self_term(S, a, k, dist(xc, a, k, dx, dy, dz), t, dt);
         s += t;
+        ds_out[2 * static_cast<size_t>(p) + (j < nf ? 0 : 1)] = dt;   // ds_ak/dr for the force pass (this side)
     }
-    for (int q = S.rev_off[a]; q < S.rev_off[a + 1]; q++) {
-        const int k = S.pairs[S.rev_pair[q]].x;
-        self_term(S, a, k, dist(xc, a, k, dx, dy, dz), t, dt);
-        s += t;
+    s = warp_sum(s) + 1.0 / (2.0 * S.eps_s * S.R[a]);
+    if (lane == 0) {
+        s_out[w] = s;
+        alpha_out[w] = S.tau / (2.0 * s);
+        eself[w] = 332.0 * S.q[a] * S.q[a] * s;
     }
-    s_out[idx] = s;
-    alpha_out[idx] = S.tau / (2.0 * s);
-    eself[idx] = 332.0 * S.q[a] * S.q[a] * s;
 }
 
 // (b) pairwise GB (Eq. 7, reading E4) + shifted 6-12 vdW (Eqs. 8-10, reading E5): energies, dE/dr at fixed
@@ -123,50 +149,63 @@ __global__ void k_em_pair(Sys S, const double* __restrict__ x, int nconf, const 
     dal[idx] = make_double2(dEdf2 * df2da * aj, dEdf2 * df2da * ai);
 }
 
-// c_a = dE/ds_a = 332 q_a^2 + (sum of dE_GB/dalpha_a over a's pairs) * dalpha_a/ds_a (reading E6)
+// c_a = dE/ds_a = 332 q_a^2 + (sum of dE_GB/dalpha_a over a's pairs) * dalpha_a/ds_a (reading E6); warp per atom
 __global__ void k_em_chain(Sys S, int nconf, const double* __restrict__ s, const double2* __restrict__ dal,
                            double* cfac)
 {
-    const long long idx = blockIdx.x * static_cast<long long>(blockDim.x) + threadIdx.x;
-    if (idx >= static_cast<long long>(nconf) * S.n) return;
-    const int c = static_cast<int>(idx / S.n), a = static_cast<int>(idx % S.n);
+    const long long w = (blockIdx.x * static_cast<long long>(blockDim.x) + threadIdx.x) >> 5;
+    const int lane = threadIdx.x & 31;
+    if (w >= static_cast<long long>(nconf) * S.n) return;
+    const int c = static_cast<int>(w / S.n), a = static_cast<int>(w % S.n);
     const double2* dc = dal + static_cast<size_t>(c) * S.np;
+    const int nf = S.fwd_off[a + 1] - S.fwd_off[a], nn = nf + S.rev_off[a + 1] - S.rev_off[a];
     double G = 0.0;
-    for (int p = S.fwd_off[a]; p < S.fwd_off[a + 1]; p++) G += dc[p].x;
-    for (int q = S.rev_off[a]; q < S.rev_off[a + 1]; q++) G += dc[S.rev_pair[q]].y;
-    const double sa = s[idx];
-    cfac[idx] = 332.0 * S.q[a] * S.q[a] + G * (-S.tau / (2.0 * sa * sa));
+    for (int j = lane; j < nn; j += 32) {
+        int p, k;
+        neighbour(S, a, nf, j, p, k);
+        G += j < nf ? dc[p].x : dc[p].y;
+    }
+    G = warp_sum(G);
+    if (lane == 0) {
+        const double sa = s[w];
+        cfac[w] = 332.0 * S.q[a] * S.q[a] + G * (-S.tau / (2.0 * sa * sa));
+    }
 }
 
-// (c) forces: F_a = -sum over a's pairs of (dE/dr_p + c_a ds_ak/dr + c_k ds_ka/dr) (x_a - x_k)/r
+// (c) forces: F_a = -sum over a's pairs of (dE/dr_p + c_a ds_ak/dr + c_k ds_ka/dr) (x_a - x_k)/r; warp per atom
 __global__ void k_em_force(Sys S, const double* __restrict__ x, int nconf, const double* __restrict__ dEdr,
-                           const double* __restrict__ cfac, double* f)
+                           const double2* __restrict__ dsd, const double* __restrict__ cfac, double* f)
 {
-    const long long idx = blockIdx.x * static_cast<long long>(blockDim.x) + threadIdx.x;
-    if (idx >= static_cast<long long>(nconf) * S.n) return;
-    const int c = static_cast<int>(idx / S.n), a = static_cast<int>(idx % S.n);
+    const long long w = (blockIdx.x * static_cast<long long>(blockDim.x) + threadIdx.x) >> 5;
+    const int lane = threadIdx.x & 31;
+    if (w >= static_cast<long long>(nconf) * S.n) return;
+    const int c = static_cast<int>(w / S.n), a = static_cast<int>(w % S.n);
     const double* xc = x + static_cast<size_t>(c) * S.n * 3;
     const double* dr = dEdr + static_cast<size_t>(c) * S.np;
     const double* cf = cfac + static_cast<size_t>(c) * S.n;
     const double ca = cf[a];
-    double fx = 0.0, fy = 0.0, fz = 0.0, dx, dy, dz, t, dak, dka;
-    auto add = [&](int p, int k) {
+    const int nf = S.fwd_off[a + 1] - S.fwd_off[a], nn = nf + S.rev_off[a + 1] - S.rev_off[a];
+    const double2* dsc = dsd + static_cast<size_t>(c) * S.np;
+    double fx = 0.0, fy = 0.0, fz = 0.0, dx, dy, dz;
+    for (int j = lane; j < nn; j += 32) {
+        int p, k;
+        neighbour(S, a, nf, j, p, k);
         const double r = dist(xc, a, k, dx, dy, dz);
-        self_term(S, a, k, r, t, dak);
-        self_term(S, k, a, r, t, dka);
+        const double2 ds = dsc[p];   // (ds_ij/dr, ds_ji/dr) of pair p = (i, j), from k_em_self
+        const double dak = j < nf ? ds.x : ds.y, dka = j < nf ? ds.y : ds.x;
         const double de = (dr[p] + ca * dak + cf[k] * dka) / r;
         fx -= de * dx;
         fy -= de * dy;
         fz -= de * dz;
-    };
-    for (int p = S.fwd_off[a]; p < S.fwd_off[a + 1]; p++) add(p, S.pairs[p].y);
-    for (int q = S.rev_off[a]; q < S.rev_off[a + 1]; q++) {
-        const int p = S.rev_pair[q];
-        add(p, S.pairs[p].x);
     }
-    f[3 * idx] = fx;
-    f[3 * idx + 1] = fy;
-    f[3 * idx + 2] = fz;
+    fx = warp_sum(fx);
+    fy = warp_sum(fy);
+    fz = warp_sum(fz);
+    if (lane == 0) {
+        f[3 * w] = fx;
+        f[3 * w + 1] = fy;
+        f[3 * w + 2] = fz;
+    }
 }
 
 // per conformation: E_self = sum over atoms, E_GB and E_vdw = sums over pairs (fixed-order reduction)
@@ -203,7 +242,7 @@ struct dock_em_ctx {
     em::Sys S{};
     void* blob = nullptr;          // device copy of every parameter array
     double *s = nullptr, *alpha = nullptr, *eself = nullptr, *dEdr = nullptr, *cfac = nullptr;
-    double2 *e_pair = nullptr, *dal = nullptr;
+    double2 *e_pair = nullptr, *dal = nullptr, *dsd = nullptr;
     double *d_x = nullptr, *d_e = nullptr, *d_f = nullptr;
     int cap_conf = 0;
     cudaEvent_t ev[2] = {nullptr, nullptr};
@@ -262,11 +301,12 @@ bool fetch(const T* src, size_t n, std::vector<T>& dst, int device)
 
 void em_free(dock_em_ctx* c)
 {
-    void* bufs[] = {c->blob, c->s, c->alpha, c->eself, c->dEdr, c->cfac, c->e_pair, c->dal, c->d_x, c->d_e, c->d_f};
+    void* bufs[] = {c->blob, c->s, c->alpha, c->eself, c->dEdr, c->cfac, c->e_pair, c->dal, c->dsd,
+                    c->d_x,  c->d_e, c->d_f};
     for (void* b : bufs)
         if (b) cudaFree(b);
     c->s = c->alpha = c->eself = c->dEdr = c->cfac = c->d_x = c->d_e = c->d_f = nullptr;
-    c->e_pair = c->dal = nullptr;
+    c->e_pair = c->dal = c->dsd = nullptr;
     c->blob = nullptr;
 }
 
@@ -455,6 +495,7 @@ dock_status dock_em_eval(dock_em_ctx* ctx, const double* xyz, int n_conf, double
         ECU(cudaMalloc(&ctx->dEdr, sizeof(double) * cp));
         ECU(cudaMalloc(&ctx->e_pair, sizeof(double2) * cp));
         ECU(cudaMalloc(&ctx->dal, sizeof(double2) * cp));
+        ECU(cudaMalloc(&ctx->dsd, sizeof(double2) * cp));
         ECU(cudaMalloc(&ctx->d_x, sizeof(double) * cn * 3));
         ECU(cudaMalloc(&ctx->d_e, sizeof(double) * 3 * n_conf));
         ECU(cudaMalloc(&ctx->d_f, sizeof(double) * cn * 3));
@@ -471,13 +512,16 @@ dock_status dock_em_eval(dock_em_ctx* ctx, const double* xyz, int n_conf, double
     const long long na = (long long)n_conf * n, npc = (long long)n_conf * np;
     const int B = 128;
     ECU(cudaEventRecord(ctx->ev[0], st));
-    em::k_em_self<<<(unsigned)((na + B - 1) / B), B, 0, st>>>(S, dx, n_conf, ctx->s, ctx->alpha, ctx->eself);
+    const long long naw = na * 32;   // warp per (conformation, atom)
+    em::k_em_self<<<(unsigned)((naw + B - 1) / B), B, 0, st>>>(S, dx, n_conf, ctx->s, ctx->alpha, ctx->eself,
+                                                                ctx->dsd);
     if (np > 0)
         em::k_em_pair<<<(unsigned)((npc + B - 1) / B), B, 0, st>>>(S, dx, n_conf, ctx->alpha, ctx->e_pair, ctx->dEdr,
                                                                  ctx->dal);
     if (df) {
-        em::k_em_chain<<<(unsigned)((na + B - 1) / B), B, 0, st>>>(S, n_conf, ctx->s, ctx->dal, ctx->cfac);
-        em::k_em_force<<<(unsigned)((na + B - 1) / B), B, 0, st>>>(S, dx, n_conf, ctx->dEdr, ctx->cfac, df);
+        em::k_em_chain<<<(unsigned)((naw + B - 1) / B), B, 0, st>>>(S, n_conf, ctx->s, ctx->dal, ctx->cfac);
+        em::k_em_force<<<(unsigned)((naw + B - 1) / B), B, 0, st>>>(S, dx, n_conf, ctx->dEdr, ctx->dsd, ctx->cfac,
+                                                                     df);
     }
     em::k_em_energy<<<n_conf, 256, 0, st>>>(S.n, S.np, ctx->eself, ctx->e_pair, de);
     ECU(cudaGetLastError());
