@@ -9,6 +9,9 @@ python -c "import __graft_entry__ as e; e.build()" > gpurun_out/build_${TAG}.log
 echo "== bench prod"; timeout 900 python bench.py > gpurun_out/bench_${TAG}_prod.json 2> gpurun_out/bench_${TAG}_prod.err; echo "rc=$?"
 echo "== bench c64"; timeout 600 python bench.py --config c64 --no-cpu-baseline > gpurun_out/bench_${TAG}_c64.json 2> gpurun_out/bench_${TAG}_c64.err; echo "rc=$?"
 echo "== bench large shard"; timeout 900 python bench.py --config large --rotations 8750 --steps 3 --warmup 3 --no-cpu-baseline --no-e2e > gpurun_out/bench_${TAG}_large.json 2> gpurun_out/bench_${TAG}_large.err; echo "rc=$?"
+echo "== shard times (single-GPU projection input)"; timeout 600 python scripts/shard_times.py > gpurun_out/shard_times_${TAG}_prod.json; timeout 900 python scripts/shard_times.py --config large --rotations 8750 --steps 3 > gpurun_out/shard_times_${TAG}_large.json; tail -c 400 gpurun_out/shard_times_${TAG}_prod.json
+echo "== host gaps"; python scripts/host_gaps.py > gpurun_out/host_gaps_${TAG}.json
+echo "== EM bench"; python scripts/bench_em.py > gpurun_out/em_bench_${TAG}.json
 echo "== launch list prod"
 timeout 900 ncu --metrics gpu__time_duration.sum --clock-control none --csv --log-file gpurun_out/launches_${TAG}_prod.csv \
     python bench.py --steps 2 --warmup 1 --no-e2e --no-cpu-baseline --no-alt > gpurun_out/launches_${TAG}_prod.log 2>&1; echo "rc=$?"
