@@ -808,14 +808,14 @@ dock_status sp_prepare(dock_ctx* ctx, int m, const dock_probe_desc* probes, int 
 }
 
 // Cost model of the engine choice (auto), per SM-clock rates measured on B200: the sparse
-// engine gathers ~6 values (one per occupied voxel and translation); the tensor-core engine executes ~3000
+// engine gathers ~7.5 values (one per occupied voxel and translation); the tensor-core engine executes ~3000
 // bf16 MACs (K-steps of 16 per rotation and translation, its bf16x3 split and padding included); the FFMA
 // engine ~170 FP32 FMAs.
 bool sp_better(dock_ctx* ctx, const SpCall& sc, int m, int n_units)
 {
     if (!sc.ok) return false;
     const double ncell = (double)ctx->nx * ctx->ny * ctx->nz;
-    const double sparse = sc.terms * ncell / 6.0;
+    const double sparse = sc.terms * ncell / 7.5;
     int v = 0, G = 0;
     double dense;
     if (plan_tc_launch(ctx, m, tc::ROT, &v, &G))

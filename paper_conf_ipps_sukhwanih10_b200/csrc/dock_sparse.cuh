@@ -20,8 +20,9 @@
 //
 // k_corr_sparse: one CTA = (group of RB rotations of one probe, range of columns of TX x TY x nz translations).
 // The producer warp streams z-planes of every atom grid G_a (TMA, one box [TY+m-1][TX+m-1] per atom and
-// plane) through a ring of NPL plane slots; 8 consumer warps = TY rows x 2 plane groups of ZT planes per
-// step (ZT = 2 for 64-translation rows, else 1); lane j owns the translations x0 + j + 32 i (i < XTS) of
+// plane) through a ring of NPL plane slots; 16 consumer warps = TY rows x 2 plane groups of ZT planes per
+// step (ZT = 2 for 64-translation rows, else 1) x 2 halves of the item's rotations (4 per warp: 4 warps per
+// scheduler hide the gather latency); lane j owns the translations x0 + j + 32 i (i < XTS) of
 // its row in each of its planes, so every shared-memory read of a warp is 32 consecutive words
 // (conflict-free for any voxel offset).  Per rotation the occupied voxels' terms are gathered from the
 // ring, then the per-warp top-32 key lists of the FFMA engine take the scores (no score grid in HBM);
@@ -37,7 +38,9 @@ using dk::KEY_MAX;
 constexpr int RB = 8;                     // rotations per item (accumulated side by side: independent chains)
 constexpr int TY = 4;                     // translation rows per column
 constexpr int NPG = 2;                    // plane groups per step (warps = TY rows x NPG groups)
-constexpr int NWC = TY * NPG;             // consumer warps
+constexpr int RSPLIT = 2;                 // rotation halves: two warps share a (row, plane group), RB/2 rotations each
+constexpr int RBW = RB / RSPLIT;          // rotations per warp
+constexpr int NWC = TY * NPG * RSPLIT;    // consumer warps (16: 4 per scheduler)
 // ZT = planes per warp and step (a template parameter): 2 for the narrow 64-translation rows when the plane
 // ring fits (more values per term decode and per gate), else 1; a step advances NPG * ZT planes
 constexpr int NTHREADS = (NWC + 1) * 32;  // + 1 TMA producer warp
@@ -329,8 +332,8 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
                                          // (branch-free loop)
     __shared__ int s_dterm[TMAX * RB];   // [term][rotation]: direct term (vx | vy << 8 | vz << 16 | term << 24) or -1
     __shared__ int s_tmax, s_ndirect;    // most occupied voxels of a rotation of the group; direct terms in the group
-    __shared__ unsigned long long s_lst[NWC][RB][32];   // per warp and rotation: sorted top-32 keys (one per lane)
-    __shared__ float2 s_th[NWC][RB];                     // per list: score bound and t_lin of its 32nd key
+    __shared__ unsigned long long s_lst[NWC][RBW][32];   // per warp and rotation: sorted top-32 keys (one per lane)
+    __shared__ float2 s_th[NWC][RBW];                     // per list: score bound and t_lin of its 32nd key
 
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     const int grp = blockIdx.x / a.G, reg = blockIdx.x % a.G;
@@ -411,11 +414,11 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
     }
 
     // ---------------- consumers: warp = (row ry, plane group pg: planes pg * ZT .. pg * ZT + ZT - 1 of a step)
-    const int ry = warp % TY, pg = warp / TY;
+    const int ry = warp % TY, pg = (warp / TY) % NPG, rbase = (warp / (TY * NPG)) * RBW;   // rotations rbase..+RBW-1
     unsigned long long(*lists)[32] = s_lst[warp];
 #pragma unroll
-    for (int r = 0; r < RB; r++) lists[r][lane] = KEY_MAX;
-    if (lane < RB) s_th[warp][lane] = make_float2(__int_as_float(0x7f800000), __uint_as_float(0xffffffffu));
+    for (int r = 0; r < RBW; r++) lists[r][lane] = KEY_MAX;
+    if (lane < RBW) s_th[warp][lane] = make_float2(__int_as_float(0x7f800000), __uint_as_float(0xffffffffu));
     __syncwarp();
     const uint32_t lane_base = dk::smem_u32(ring) + 4u * static_cast<uint32_t>(ry * a.TXB + lane);
     const uint32_t ring_bytes = static_cast<uint32_t>(npl * slot_bytes);
@@ -462,11 +465,11 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
                 // term-outer, rotation-inner, branch-free: the RB rotations' gathers are independent (weight 1 for
                 // a single-atom voxel, 0 for an absent or multi-atom term: fma(1, g, acc) == acc + g exactly);
                 // term 0 initialises the accumulators
-                float acc[RB][V];
+                float acc[RBW][V];
                 if (tmax > 0) {
 #pragma unroll
-                    for (int r = 0; r < RB; r++) {
-                        const int4 term = s_term[r];
+                    for (int r = 0; r < RBW; r++) {
+                        const int4 term = s_term[rbase + r];
                         const float wt = __int_as_float(term.z);
 #pragma unroll
                         for (int j = 0; j < ZT; j++) {
@@ -479,15 +482,15 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
                     }
                 } else {   // a probe without atoms scores 0 everywhere
 #pragma unroll
-                    for (int r = 0; r < RB; r++)
+                    for (int r = 0; r < RBW; r++)
 #pragma unroll
                         for (int v = 0; v < V; v++) acc[r][v] = 0.0f;
                 }
 #pragma unroll 1
                 for (int t = 1; t < tmax; t++) {
 #pragma unroll
-                    for (int r = 0; r < RB; r++) {
-                        const int4 term = s_term[t * RB + r];
+                    for (int r = 0; r < RBW; r++) {
+                        const int4 term = s_term[t * RB + rbase + r];
                         const float wt = __int_as_float(term.z);
 #pragma unroll
                         for (int j = 0; j < ZT; j++) {
@@ -505,13 +508,13 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
 #pragma unroll 1
                     for (int t = 0; t < tmax; t++) {
 #pragma unroll
-                        for (int r = 0; r < RB; r++) {
-                            const int code = s_dterm[t * RB + r];
+                        for (int r = 0; r < RBW; r++) {
+                            const int code = s_dterm[t * RB + rbase + r];
                             if (code >= 0) {
 #pragma unroll
                                 for (int j = 0; j < ZT; j++) {
                                     const Vec<XTS> d = sp_direct<XTS>(
-                                        a.dw + (static_cast<size_t>(gr.slot0 + r) * TMAX + (code >> 24)) * a.P, a.P,
+                                        a.dw + (static_cast<size_t>(gr.slot0 + rbase + r) * TMAX + (code >> 24)) * a.P, a.P,
                                         a.rec, a.rXp, a.rYp, a.rZp, z0w + j + ((code >> 16) & 0xff),
                                         y + ((code >> 8) & 0xff), xb + (code & 0xff), (vmask >> (j * XTS)) & xmask);
 #pragma unroll
@@ -523,9 +526,9 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
                 }
                 if constexpr (GRID) {
 #pragma unroll
-                    for (int r = 0; r < RB; r++) {
-                        if (r < nrot) {
-                            float* out = a.grid + static_cast<size_t>(grp + r) * a.nx * a.ny * a.nz + tbase;
+                    for (int r = 0; r < RBW; r++) {
+                        if (rbase + r < nrot) {
+                            float* out = a.grid + static_cast<size_t>(grp + rbase + r) * a.nx * a.ny * a.nz + tbase;
 #pragma unroll
                             for (int v = 0; v < V; v++)
                                 if ((vmask >> v) & 1u) out[(v / XTS) * plane_stride + 32 * (v % XTS)] = acc[r][v];
@@ -536,7 +539,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
                     // precede the list's 32nd key (tbase is the smallest t_lin of the lane); one warp vote for all
                     unsigned pass = 0;
 #pragma unroll
-                    for (int r = 0; r < RB; r++) {
+                    for (int r = 0; r < RBW; r++) {
                         const float2 thr = s_th[warp][r];
                         float mn;
                         if (vfull) {
@@ -549,12 +552,12 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
                             for (int v = 0; v < V; v++) mn = ((vmask >> v) & 1u) ? fminf(mn, acc[r][v]) : mn;
                         }
                         const bool any = mn < thr.x || (mn == thr.x && tbase < __float_as_uint(thr.y));
-                        pass |= (any && r < nrot) ? (1u << r) : 0u;
+                        pass |= (any && rbase + r < nrot) ? (1u << r) : 0u;
                     }
                     pass = __reduce_or_sync(FULL, pass);
                     if (pass) {
 #pragma unroll
-                        for (int r = 0; r < RB; r++) {
+                        for (int r = 0; r < RBW; r++) {
                             if ((pass >> r) & 1u) {
                                 Vec<V> av;
 #pragma unroll
@@ -590,9 +593,9 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
         // ---------------- item end: publish bound + surviving keys of each warp list (as dk::k_corr)
         const int nx = a.nx, ny = a.ny, nz = a.nz;
 #pragma unroll 1
-        for (int rr = 0; rr < nrot; rr++) {
+        for (int rr = 0; rr < RBW && rbase + rr < nrot; rr++) {
             {
-                const int slot = gr.slot0 + rr;
+                const int slot = gr.slot0 + rbase + rr;
                 const unsigned long long key = lists[rr][lane];
                 const uint32_t t = static_cast<uint32_t>(key & 0xffffffffu);
                 const unsigned long long k31 = dk::shfl_u64(key, 31);
