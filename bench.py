@@ -56,6 +56,7 @@ def parse():
                          "sparse (FP32 sparse-ligand gathers)")
     ap.add_argument("--no-alt", action="store_true", help="skip the secondary measurement of the other engine")
     ap.add_argument("--tc-epi", type=int, default=0, choices=[0, 4, 8, 16], help="tcgen05 epilogue warps (0 auto)")
+    ap.add_argument("--tc-chunk", type=int, default=0, help="tcgen05 tiles per scheduled chunk (0 auto)")
     ap.add_argument("--tc-variant", type=int, default=0, choices=[0, 1, 2],
                     help="tcgen05 kernel: 0 auto, 1 = resident receptor boxes (P <= 4), 2 = streamed (group, z-plane) units")
     return ap.parse_args()
@@ -237,7 +238,8 @@ def roofline(pk, pk_kind, info, c, flops_launch, corr_ms, ms_step, units_local):
         ach = gbytes / (corr_ms / 1000.0) / 1e9
         peak = n_sms * 128 * sm_max * 1e6 / 1e9
         xts = max(1, int(info.get("sp_row_last", 128)) // 32)
-        return {"bound": "smem", "engine": "sparse ligand (fp32 gathers)", "kernel": f"k_corr_sparse<{xts},false>",
+        zt = max(1, int(info.get("sp_zt_last", 1)))
+        return {"bound": "smem", "engine": "sparse ligand (fp32 gathers)", "kernel": f"k_corr_sparse<{xts},{zt},false>",
                 "achieved": ach, "peak": peak, "unit": "GB/s", "frac": ach / peak, "traffic": None,
                 "peak_source": f"{n_sms} SMs x 128 B/clk shared-memory loads x {sm_max:.0f} MHz (sm_max_mhz, "
                                f"MEASURED_PEAKS.json: {pk_kind})",
@@ -302,8 +304,11 @@ def run_ours(args):
     D.dock_set_tuning(ctx, D.DOCK_TUNE_ENGINE, ENG[args.engine])
     D.dock_set_tuning(ctx, D.DOCK_TUNE_TC_VARIANT, args.tc_variant)
     D.dock_set_tuning(ctx, 6, args.tc_epi)   # DOCK_TUNE_TC_EPILOGUE_WARPS
+    D.dock_set_tuning(ctx, D.DOCK_TUNE_TC_CHUNK, args.tc_chunk)
     probes_dev = [{"xyz": torch.from_numpy(p.xyz).to(dev), "coef": torch.from_numpy(p.coef).to(dev), "m": p.m}
                   for p in probes]
+    # probe descriptors marshalled once (the probe arrays stay where they are: device here, host in e2e)
+    probes_dev = D.dock_probes(ctx, probes_dev)
     rot_dev = torch.from_numpy(rot).to(dev)
     if world > 1:
         pg = parallel.pose_gather(n_units, k, dev)   # preallocated all-gather buffer; poses land in its slot
@@ -381,11 +386,12 @@ def run_ours(args):
         h2d = rot.nbytes + sum(p.xyz.nbytes + p.coef.nbytes for p in probes) + 4 * (len(probes) + 1)
         d2h = n_units * k * 16
         out2 = pg.slot if world > 1 else torch.empty((e - b, k, 4), dtype=torch.int32, device=dev)
+        probes_host = D.dock_probes(ctx, probes)   # host arrays: staged and copied H2D inside every call
 
         def step_e2e():
             # host numpy inputs (pinned staging + H2D inside the call), device poses, D2H read of the result
             if e > b:
-                D.dock_probe_batch(ctx, probes, rot, b, e, k, args.rho, out=out2)
+                D.dock_probe_batch(ctx, probes_host, rot, b, e, k, args.rho, out=out2)
             full = pg.gather() if world > 1 else out2
             if rank == 0:
                 full.cpu()
@@ -420,7 +426,9 @@ def run_ours(args):
         # capture was taken of this exact kernel build (sha256 of its SASS), else reported as stale
         with open(tp) as f:
             tj = json.load(f)
-        ent = tj.get(roof["kernel"])
+        # entries keyed "<kernel>@<config>[@r<rotations>]" (the exact bench launch), else "<kernel>"
+        key = f'{roof["kernel"]}@{args.config}' + (f"@r{args.rotations}" if args.rotations else "")
+        ent = tj.get(key) or tj.get(roof["kernel"])
         if ent and ent.get("config") == args.config and ent.get("gpus") == world:
             now = kernel_sass_sha(roof["kernel"])
             if now and ent.get("sass_sha256") == now:

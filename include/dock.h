@@ -158,7 +158,8 @@ dock_status dock_voxelize(dock_ctx* ctx, const dock_probe_desc* probe, const dou
 
 /* Tuning / introspection ------------------------------------------------------------- */
 typedef enum {
-    DOCK_TUNE_REGIONS = 1,        /* translation regions per rotation batch (0 = auto) */
+    DOCK_TUNE_REGIONS = 1,        /* translation regions per rotation batch (0 = auto; > 0 also turns off
+                                     the tcgen05 variant-1 dynamic tile scheduler) */
     DOCK_TUNE_FORCE_FALLBACK = 2, /* 1 => every rotation takes the exact full-grid fallback (tests) */
     DOCK_TUNE_CAND_CAP = 3,       /* candidates kept per rotation before overflow fallback (>= 32) */
     DOCK_TUNE_ENGINE = 4,         /* correlation engine: 0 auto (tcgen05 when eligible), 1 FP32 FFMA, 2 tcgen05,
@@ -174,16 +175,19 @@ typedef enum {
                                      z-plane) unit at a time (any P <= 32, m <= 8; 64 / 128 / 160 translations per
                                      row, chosen at init for nx).  A variant that cannot run m falls back to the
                                      other one. */
-    DOCK_TUNE_TC_EPILOGUE_WARPS = 6 /* tcgen05 epilogue warps: 0 auto (= the compiled maximum, 8), 4 or 8 (values
+    DOCK_TUNE_TC_EPILOGUE_WARPS = 6, /* tcgen05 epilogue warps: 0 auto (= the compiled maximum, 8), 4 or 8 (values
                                      above the compiled maximum are clamped to it) */
+    DOCK_TUNE_TC_CHUNK = 7        /* tcgen05 variant 1: tiles per dynamically scheduled chunk (0 = auto, 4;
+                                     1..4096); one persistent CTA per SM takes chunks from a device counter */
 } dock_tune_key;
 
 dock_status dock_set_tuning(dock_ctx* ctx, int key, int64_t value);
 
 typedef struct {
     int lanes_x, tile_x, tile_y, tile_z, n_tiles, n_stages, smem_bytes;
-    int regions_last;          /* regions used by the last dock_probe_batch */
-    int64_t items_last;        /* CTAs (rotation batch x region) launched by the last call */
+    int regions_last;          /* regions per rotation batch of the last dock_probe_batch (0: tcgen05 variant 1's
+                                  dynamic tile scheduler, DOCK_TUNE_TC_CHUNK) */
+    int64_t items_last;        /* CTAs launched by the last call's correlation */
     int64_t fallback_last;     /* rotations that took the exact fallback in the last call (valid after its sync point) */
     int64_t cand_max_last;     /* largest candidate count of one rotation in the last call (idem) */
     int64_t kernels_last;      /* kernels launched by the last call */
@@ -204,6 +208,7 @@ typedef struct {
     int sp_atom_grids_last;    /* sparse engine: atom grids G_a computed by the last call */
     int sp_row_last;           /* sparse engine: translations per column row (32 x per-lane count) */
     double sp_terms_last;      /* sparse engine: atoms summed over the units of the last call (gathers per translation) */
+    int sp_zt_last;            /* sparse engine: z planes per warp and step of the last call (1 or 2) */
 } dock_info;
 
 dock_status dock_get_info(const dock_ctx* ctx, dock_info* info);

@@ -76,11 +76,15 @@ struct dock_ctx {
     float* d_eye = nullptr;    // [P][P] identity (per-term grids)
     float* d_ones = nullptr;   // [P] ones (unweighted voxel export)
     MPlan plan[DOCK_MAX_M + 1];
+    std::vector<unsigned char> probe_dev;   // [2 n_probes] device-memory flags (xyz, coef) of the probes of
+                                            // the current call, set by validate_probes for stage_inputs
     // tcgen05 engine
     int engine = 0;            // DOCK_TUNE_ENGINE: 0 auto, 1 FFMA, 2 tensor cores, 3 FFT (comparison engine)
     DockFft* fft = nullptr;    // FFT engine state (receptor transform, plans, work buffers), created on first use
     int engine_last = 0;
     int tc_variant = 0;        // DOCK_TUNE_TC_VARIANT: 0 auto, 1 resident boxes (P <= 4), 2 streamed planes
+    int tc_chunk = 0;          // DOCK_TUNE_TC_CHUNK: tiles per scheduled chunk (variant 1), 0 = auto
+    unsigned long long* d_sched = nullptr;   // [1 + n_sms] dynamic tile scheduler counters (self-resetting)
     int tc_variant_last = 0;
     int tc_m_last = 0;
     int tc_ksteps_last = 0;    // K-steps (of 16) per translation row in the last tcgen05 launch
@@ -123,7 +127,7 @@ struct dock_ctx {
     DevBuf sp_G, sp_tv, sp_ts, sp_nt, sp_dw, sp_slot_atoms;
     CUtensorMap sp_tmap;
     int sp_natoms_last = 0;           // atom grids of the last sparse call
-    int sp_tx_last = 0;
+    int sp_tx_last = 0, sp_zt_last = 0;
     double sp_terms_last = 0;         // occupied voxels summed over the units of the last sparse call
     // tuning
     int regions_override = 0;
@@ -470,7 +474,10 @@ dock_status stage_inputs(dock_ctx* ctx, const dock_probe_desc* probes, int n_pro
 {
     // One pinned staging block [fb args][off][gather table][rot (host)][host xyz][host coef] goes up in a
     // single H2D copy; one gather kernel then assembles all probes' atoms (device-resident probe arrays are
-    // read in place).  The host part stays short and never waits for the GPU (staging ring).
+    // read in place).  The host part stays short and never waits for the GPU (staging ring).  The probes'
+    // memory kinds are those validate_probes recorded for this call.
+    if (ctx->probe_dev.size() != 2 * (size_t)n_probes)
+        return fail(ctx, DOCK_E_INVALID_ARG, "internal: probes not validated");
     const int P = ctx->P;
     std::vector<int> off(n_probes + 1, 0);
     for (int i = 0; i < n_probes; i++) off[i + 1] = off[i] + probes[i].n_atoms;
@@ -502,9 +509,7 @@ dock_status stage_inputs(dock_ctx* ctx, const dock_probe_desc* probes, int n_pro
         t.off = off[i];
         if (pr.n_atoms > 0) {
             const size_t bx = sizeof(double) * 3 * pr.n_atoms, bc = sizeof(float) * P * pr.n_atoms;
-            bool xd = false, cd = false;
-            PTR_KIND(xd, pr.xyz, "probe xyz");
-            PTR_KIND(cd, pr.coef, "probe coef");
+            const bool xd = ctx->probe_dev[2 * i], cd = ctx->probe_dev[2 * i + 1];
             if (xd) {
                 t.xyz = pr.xyz;
             } else {
@@ -553,6 +558,7 @@ dock_status validate_probes(dock_ctx* ctx, const dock_probe_desc* probes, int n_
 {
     if (!probes || n_probes < 1) return fail(ctx, DOCK_E_INVALID_ARG, "no probes");
     int m = probes[0].m;
+    ctx->probe_dev.assign(2 * (size_t)n_probes, 0);
     for (int i = 0; i < n_probes; i++) {
         const dock_probe_desc& p = probes[i];
         if (p.n_atoms < 0) return fail(ctx, DOCK_E_INVALID_ARG, "probe %d: n_atoms < 0", i);
@@ -564,6 +570,8 @@ dock_status validate_probes(dock_ctx* ctx, const dock_probe_desc* probes, int n_
         bool xd = false, cd = false;
         PTR_KIND(xd, p.xyz, "probe xyz");
         PTR_KIND(cd, p.coef, "probe coef");
+        ctx->probe_dev[2 * i] = xd;
+        ctx->probe_dev[2 * i + 1] = cd;
         if (!xd && p.n_atoms > 0) {
             for (int j = 0; j < 3 * p.n_atoms; j++)
                 if (!std::isfinite(p.xyz[j])) return fail(ctx, DOCK_E_INVALID_ARG, "probe %d: non-finite xyz", i);
@@ -659,7 +667,23 @@ tc::TcArgs tc_args(dock_ctx* ctx, int m, int v, int n_slots, int G, const unsign
     a.wstages = tp.wstages;
     a.nepi = ctx->tc_nepi > 0 ? std::min(tc::NEPI_MAX, ctx->tc_nepi) : tc::NEPI_MAX;
     a.trace = ctx->d_trace;
+    // variant 1 (one CTA per SM: >= 116 KB shared memory, all 512 TMEM columns): a persistent CTA per SM takes
+    // chunks of tc_chunk tiles of one rotation block from a device counter.  Per-tile cost varies with the
+    // receptor region (top-k insertions), so static splits leave SMs idle at the end (measured: CTA lifetimes
+    // 1.05-2.05 ms for equal tile counts at 1008 rotations); region mode also quantises to whole waves.  A
+    // forced region count (DOCK_TUNE_REGIONS) keeps region mode.
+    a.chunk = 0;
+    a.sched = ctx->d_sched;
+    if (v == 1 && ctx->regions_override <= 0 && ctx->d_sched) a.chunk = ctx->tc_chunk > 0 ? ctx->tc_chunk : 4;
     return a;
+}
+
+// CTAs of a tensor-core launch over n_slots rotations.
+int64_t tc_ctas(const tc::TcArgs& a, int n_slots, int n_sms)
+{
+    const int64_t n_blocks = (n_slots + tc::ROT - 1) / tc::ROT;
+    if (a.chunk > 0) return std::min<int64_t>(n_sms, n_blocks * ((a.ntiles + a.chunk - 1) / a.chunk));
+    return n_blocks * a.G;
 }
 
 // Variant + regions for a launch over n_slots rotations; returns false if the tensor cores can't run m.
@@ -907,6 +931,7 @@ dock_status sp_run_pre(dock_ctx* ctx, const SpCall& sc, int n_slots, int64_t uni
     ctx->kernels_last++;
     ctx->sp_natoms_last = sc.n_at;
     ctx->sp_tx_last = pl.TX;
+    ctx->sp_zt_last = sc.zt;
     ctx->sp_terms_last = sc.terms;
     return DOCK_OK;
 }
@@ -1029,7 +1054,8 @@ dock_status run_grid_tc(dock_ctx* ctx, int m, int n_slots, const float* Lw, floa
     TRY(pack_weights_tc(ctx, m, v, n_slots, Lw));
     tc::TcArgs a = tc_args(ctx, m, v, n_slots, G, static_cast<const unsigned char*>(ctx->Wtc.p));
     a.grid = grid;
-    const int64_t items = n_blocks * G;
+    const int64_t items = tc_ctas(a, n_slots, ctx->n_sms);
+    if (items > 0x7fffffff || n_blocks > 0x7fffffff) return fail(ctx, DOCK_E_UNSUPPORTED, "too many work items");
     CU(launch_tc(m, v, true, ctx->tcplan[v][m], a, (int)items, ctx->stream));
     ctx->kernels_last++;
     return DOCK_OK;
@@ -1117,7 +1143,7 @@ dock_status enqueue_fb_body(dock_ctx* ctx, const FbKey& key, const dk::FbDyn* d_
                 a.grid = grid;
                 a.n_live = &ctl->n_live;
                 a.trace = nullptr;
-                CU(launch_tc(m, key.v, true, ctx->tcplan[key.v][m], a, key.G, st));
+                CU(launch_tc(m, key.v, true, ctx->tcplan[key.v][m], a, (int)tc_ctas(a, ch, ctx->n_sms), st));
             } else {
                 const int64_t nb = (ch + dk::RB - 1) / dk::RB;
                 dk::CorrArgs a = corr_args(ctx, m, ch, key.G, Lw);
@@ -1372,6 +1398,7 @@ void dock_destroy(dock_ctx* ctx)
     for (DevBuf* b : bufs)
         if (b->p) cudaFree(b->p);
     if (ctx->d_trace) cudaFree(ctx->d_trace);
+    if (ctx->d_sched) cudaFree(ctx->d_sched);
     if (ctx->fft) dock_fft_destroy(ctx->fft);
     if (ctx->d_rec) cudaFree(ctx->d_rec);
     if (ctx->d_rec_tc) cudaFree(ctx->d_rec_tc);
@@ -1502,6 +1529,13 @@ dock_status dock_init(const dock_grid_desc* g, const float* receptor, const floa
     cudaMemcpy(ctx->d_eye, eye.data(), sizeof(float) * P * P, cudaMemcpyHostToDevice);
     cudaMemcpy(ctx->d_ones, ones.data(), sizeof(float) * P, cudaMemcpyHostToDevice);
     cudaMemsetAsync(ctx->d_small, 0, 64, ctx->stream);
+    // tcgen05 dynamic tile scheduler: [CTAs done, chunks taken per segment (one per CTA <= n_sms)], zero
+    // between launches (the last CTA of each launch resets it); without it variant 1 runs region mode
+    if (cudaMalloc(&ctx->d_sched, sizeof(unsigned long long) * (ctx->n_sms + 2)) == cudaSuccess)
+        cudaMemsetAsync(ctx->d_sched, 0, sizeof(unsigned long long) * (ctx->n_sms + 2), ctx->stream);
+    else
+        ctx->d_sched = nullptr;
+    cudaGetLastError();
     if (rec_dev) {
         dk::k_count_nonfinite<<<1024, 256, 0, ctx->stream>>>(d_src, n_in, reinterpret_cast<unsigned*>(ctx->d_small));
     }
@@ -1582,6 +1616,10 @@ dock_status dock_set_tuning(dock_ctx* ctx, int key, int64_t value)
                 return fail(ctx, DOCK_E_INVALID_ARG, "epilogue warps must be 0, 4, 8 or 16");
             ctx->tc_nepi = (int)value;
             return DOCK_OK;
+        case DOCK_TUNE_TC_CHUNK:
+            if (value < 0 || value > 4096) return fail(ctx, DOCK_E_INVALID_ARG, "tc chunk must be 0..4096");
+            ctx->tc_chunk = (int)value;
+            return DOCK_OK;
         case DOCK_TUNE_CAND_CAP:
             if (value < 32 || value > (1 << 20)) return fail(ctx, DOCK_E_INVALID_ARG, "cand cap out of range");
             ctx->cand_cap = (int)value;
@@ -1640,7 +1678,10 @@ dock_status dock_get_info(const dock_ctx* ctx, dock_info* info)
     info->fb_chunk = fb_chunk(ctx, ctx->engine_last);
     info->sp_atom_grids_last = ctx->sp_natoms_last;
     info->sp_terms_last = ctx->sp_terms_last;
-    if (ctx->engine_last == ENG_SPARSE) info->sp_row_last = ctx->sp_tx_last;
+    if (ctx->engine_last == ENG_SPARSE) {
+        info->sp_row_last = ctx->sp_tx_last;
+        info->sp_zt_last = ctx->sp_zt_last;
+    }
     return DOCK_OK;
 }
 
@@ -1779,16 +1820,26 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
         ta.mu = mup;
         ta.cnt = cntp;
         ta.cand = candp;
-        const int64_t items = n_blocks * G;
+        const int64_t items = tc_ctas(ta, n_units, ctx->n_sms);
         if (items > 0x7fffffff) return fail(ctx, DOCK_E_UNSUPPORTED, "too many work items");
         if (ctx->d_trace) CU(cudaMemsetAsync(ctx->d_trace, 0, sizeof(unsigned long long) * tc::TR_N, ctx->stream));
         CU(cudaEventRecord(ctx->ev_corr[0], ctx->stream));
         CU(launch_tc(m, v, false, ctx->tcplan[v][m], ta, (int)items, ctx->stream));
         CU(cudaEventRecord(ctx->ev_corr[1], ctx->stream));
         if (ctx->d_trace) {
-            unsigned long long h[tc::TR_N];
-            CU(cudaMemcpyAsync(h, ctx->d_trace, sizeof(h), cudaMemcpyDeviceToHost, ctx->stream));
+            std::vector<unsigned long long> hv(tc::TR_N);
+            unsigned long long* h = hv.data();
+            CU(cudaMemcpyAsync(h, ctx->d_trace, sizeof(unsigned long long) * tc::TR_N, cudaMemcpyDeviceToHost,
+                               ctx->stream));
             CU(cudaStreamSynchronize(ctx->stream));
+            if (const char* f = getenv("DOCK_TC_TRACE_CTAS")) {   // per-CTA start / end / SM id dump
+                if (FILE* fp = fopen(f, "w")) {
+                    for (int i = 0; i < (int)std::min<int64_t>(items, tc::TR_MAXCTA); i++)
+                        fprintf(fp, "%d %llu %llu %llu\n", i, h[tc::TR_CTA0 + 3 * i], h[tc::TR_CTA0 + 3 * i + 1],
+                                h[tc::TR_CTA0 + 3 * i + 2]);
+                    fclose(fp);
+                }
+            }
             const double c = h[tc::TR_CTAS] ? double(h[tc::TR_CTAS]) : 1.0;
             const double e = h[tc::TR_EPI_WARPS] ? double(h[tc::TR_EPI_WARPS]) : 1.0;
             fprintf(stderr,
@@ -1796,13 +1847,19 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
                     "\"mma_total\": %.0f, \"mma_wait_tmem_empty\": %.0f, \"mma_wait_w_full\": %.0f, "
                     "\"mma_wait_rec_full\": %.0f, \"epi_total\": %.0f, \"epi_wait_tm_full\": %.0f, "
                     "\"epi_ldtm\": %.0f, \"prod_total\": %.0f, \"prod_wait_w_empty\": %.0f, "
-                    "\"prod_wait_rec_empty\": %.0f}\n",
+                    "\"prod_wait_rec_empty\": %.0f, \"span_ms\": %.4f, \"cta_ms\": %.4f, "
+                    "\"epi_wait_chunk\": %.0f, \"mma_wait_chunk\": %.0f, \"rec_wait_chunk\": %.0f, "
+                    "\"epi_publish\": %.0f, \"inserts_per_tile_lane\": %.3f}\n",
                     v, h[tc::TR_CTAS], h[tc::TR_TILES] / c, h[tc::TR_MMA_TOTAL] / c,
                     h[tc::TR_MMA_TMEMPTY] / c, h[tc::TR_MMA_WFULL] / c, h[tc::TR_MMA_RFULL] / c,
                     h[tc::TR_EPI_TOTAL] / e, h[tc::TR_EPI_TMFULL] / e, h[tc::TR_EPI_LDTM] / e,
-                    h[tc::TR_PROD_TOTAL] / c, h[tc::TR_PROD_WEMPTY] / c, h[tc::TR_PROD_REMPTY] / c);
+                    h[tc::TR_PROD_TOTAL] / c, h[tc::TR_PROD_WEMPTY] / c, h[tc::TR_PROD_REMPTY] / c,
+                    h[tc::TR_GT_END] ? (h[tc::TR_GT_END] - ~h[tc::TR_GT_START_NOT]) * 1e-6 : 0.0,
+                    h[tc::TR_GT_CTA_NS] * 1e-6 / c, h[tc::TR_EPI_CHWAIT] / e, h[tc::TR_MMA_CHWAIT] / c,
+                    h[tc::TR_REC_CHWAIT] / c, h[tc::TR_EPI_PUB] / e,
+                    h[tc::TR_TILES] ? h[tc::TR_EPI_INS] / (double(h[tc::TR_TILES]) * tc::ROT) : 0.0);
         }
-        ctx->regions_last = G;
+        ctx->regions_last = ta.chunk > 0 ? 0 : G;
         ctx->items_last = items;
     } else {
         const int G = choose_regions(ctx, n_batches);

@@ -53,6 +53,11 @@ struct TcArgs {
     int ntx, nty, ntz, ntiles;  // tiles: NTT x Q rows (y) x 1 (z)
     int G_ch;                   // channel groups of 4
     int n_slots, G, tiles_per_region;
+    int chunk;                  // variant 1: > 0 -> dynamic scheduling: persistent CTAs (one per SM) take
+                                // chunks of `chunk` tiles of one rotation block (see k_corr_tc);
+                                // 0 -> CTA = (block, region) with G regions of tiles_per_region tiles
+    unsigned long long* sched;  // [1 + gridDim.x]: CTAs done, chunks taken per segment (zero between
+                                // launches: the last CTA to finish resets them)
     int nsteps;                 // K-steps of A per tile (all passes / units, padded to whole ring stages)
     const unsigned char* W;     // [block][step][WCHUNK]
     int box_bytes;              // bytes of one receptor TMA box (variant 1: the main box; variant 2: one z-plane)
@@ -77,7 +82,24 @@ struct TcArgs {
 
 // trace counters (cycles summed over CTAs)
 enum { TR_CTAS = 0, TR_TILES, TR_MMA_TOTAL, TR_MMA_TMEMPTY, TR_MMA_WFULL, TR_MMA_RFULL, TR_EPI_TOTAL, TR_EPI_TMFULL,
-       TR_EPI_LDTM, TR_PROD_TOTAL, TR_PROD_WEMPTY, TR_PROD_REMPTY, TR_EPI_WARPS, TR_N = 16 };
+       TR_EPI_LDTM, TR_PROD_TOTAL, TR_PROD_WEMPTY, TR_PROD_REMPTY, TR_EPI_WARPS,
+       TR_GT_START_NOT = 13,   // max over CTAs of ~(globaltimer at start): ~ = the earliest start (ns)
+       TR_GT_END = 14,         // max over CTAs of globaltimer at exit
+       TR_GT_CTA_NS = 15,      // sum over CTAs of their lifetime (ns)
+       TR_EPI_CHWAIT = 16,     // epilogue / MMA / receptor producer: waits for the next chunk (cycles)
+       TR_MMA_CHWAIT = 17,
+       TR_REC_CHWAIT = 18,
+       TR_EPI_PUB = 19,        // epilogue: publishing lists (cycles)
+       TR_EPI_INS = 20,        // epilogue: list insertions (all lanes)
+       TR_CTA0 = 24,           // per CTA (blockIdx.x < TR_MAXCTA): start, end (globaltimer), SM id
+       TR_MAXCTA = 1024,
+       TR_N = TR_CTA0 + 3 * TR_MAXCTA };
+__device__ __forceinline__ unsigned long long gtimer()
+{
+    unsigned long long t;
+    asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
+    return t;
+}
 
 // mbarrier wait that adds its duration to `acc` when tracing
 __device__ __forceinline__ void twait(uint64_t* bar, unsigned parity, bool tr, long long& acc)
@@ -206,7 +228,8 @@ __device__ __forceinline__ void list_insert(unsigned long long (&L)[LIST], unsig
 // into the per-thread exact top-LIST list; GRID writes the chunk to the score grid instead.
 template <bool GRID>
 __device__ __forceinline__ void epi_chunk(const uint32_t (&v)[32], unsigned long long (&lst)[LIST], float& th,
-                                          uint32_t& th_t, uint32_t tbase, int c0, int jmax, float* grid_row)
+                                          uint32_t& th_t, uint32_t tbase, int c0, int jmax, float* grid_row,
+                                          unsigned* nins = nullptr)
 {
     if constexpr (GRID) {
 #pragma unroll
@@ -231,6 +254,7 @@ __device__ __forceinline__ void epi_chunk(const uint32_t (&v)[32], unsigned long
                 if (sv <= th) {
                     const unsigned long long key = dk::make_key(sv, tbase + c0 + j);
                     if (key < lst[LIST - 1]) {
+                        if (nins) ++*nins;
                         list_insert(lst, key);
                         th = dk::key_score_bound(static_cast<uint32_t>(lst[LIST - 1] >> 32));
                         th_t = static_cast<uint32_t>(lst[LIST - 1] & 0xffffffffu);
@@ -288,7 +312,7 @@ __device__ __forceinline__ void epi_tile(const TcArgs& a, uint32_t tmem, uint64_
                                          int nclass, int lane, int slot, bool rot_ok, int tx, int ty, int tz,
                                          unsigned long long (&lst)[LIST], float& th, uint32_t& th_t, bool tr,
                                          long long& tw0, long long& tw1, uint64_t* row_full = nullptr,
-                                         unsigned row_ph = 0)
+                                         unsigned row_ph = 0, unsigned* nins = nullptr)
 {
     constexpr int NCH = NTT / 32;
     const int x0 = tx * NTT;
@@ -321,8 +345,8 @@ __device__ __forceinline__ void epi_tile(const TcArgs& a, uint32_t tmem, uint64_
             if (lane == 0) dk::mbar_arrive(&tm_empty[q]);
             if (!row_ok) continue;
             float* grow = GRID ? a.grid + static_cast<size_t>(slot) * a.nx * a.ny * a.nz + tbase : nullptr;
-            epi_chunk<GRID>(v0, lst, th, th_t, tbase, c0, min(32, a.nx - x0 - c0), grow);
-            epi_chunk<GRID>(v1, lst, th, th_t, tbase, c1, min(32, a.nx - x0 - c1), grow);
+            epi_chunk<GRID>(v0, lst, th, th_t, tbase, c0, min(32, a.nx - x0 - c0), grow, nins);
+            epi_chunk<GRID>(v1, lst, th, th_t, tbase, c1, min(32, a.nx - x0 - c1), grow, nins);
             continue;
         }
 #pragma unroll 1
@@ -396,22 +420,49 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
     constexpr uint32_t ROWTYP = static_cast<uint32_t>(Q + M - 1) * ROW16P;
     static_assert(Q * NT <= 512, "TMEM has 512 columns");
     extern __shared__ __align__(128) unsigned char smem[];   // TMA destinations: 128 B; no-swizzle UMMA operands: 16 B
-    __shared__ uint64_t bars[2 * 2 + 2 * WSTAGES + 2 * Q];
+    constexpr int NCR = 4;                     // chunk ring: the weight producer posts, the other roles take
+    __shared__ uint64_t bars[2 * 2 + 2 * WSTAGES + 2 * Q + 2 * NCR];
     __shared__ uint32_t tmem_base_s;
+    __shared__ long long s_cg[NCR];            // chunk: first (block, tile) pair g = block * ntiles + tile
+    __shared__ int s_cn[NCR];                  // chunk: tiles (0 = no more work)
     uint64_t* rec_full = bars;
     uint64_t* rec_empty = bars + 2;
     uint64_t* w_full = bars + 4;
     uint64_t* w_empty = w_full + WSTAGES;
     uint64_t* tm_full = w_empty + WSTAGES;   // [Q]: row q accumulated (the staircase finishes rows one by one)
     uint64_t* tm_empty = tm_full + Q;        // [Q]: row q drained, so the next tile restarts row by row
+    uint64_t* ch_full = tm_empty + Q;        // [NCR]: chunk posted
+    uint64_t* ch_empty = ch_full + NCR;      // [NCR]: chunk taken by the MMA, receptor and epilogue roles
 
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
-    const int block = blockIdx.x / a.G, region = blockIdx.x % a.G;
     const int n_eff = a.n_live ? min(a.n_slots, static_cast<int>(*a.n_live)) : a.n_slots;
-    if (block * ROT >= n_eff) return;   // uniform: a dead block of the device-driven fallback
-    const int tile_begin = region * a.tiles_per_region;
-    const int tile_end = min(a.ntiles, tile_begin + a.tiles_per_region);
-    const int n_tiles = tile_end - tile_begin;
+    const long long live_blocks = (n_eff + ROT - 1) / ROT;
+    // Work: a sequence of chunks (g, n) = n consecutive tiles of one rotation block starting at the (block,
+    // tile) pair g = block * ntiles + tile.  Region mode: the one chunk (block, region) of this CTA.  Dynamic
+    // mode: chunk c = (block c / cpb, tiles [(c % cpb) chunk, ..)), c in [0, n_chunks) split into S =
+    // gridDim.x contiguous segments with one counter each.  A CTA takes the chunks of its own segment in
+    // order (a contiguous range, so its top-k lists live long: a list restart costs a burst of insertions),
+    // then helps the next segments that still have chunks: CTAs whose tiles are cheaper (per-tile cost
+    // varies with the receptor region through the epilogue's insertions) take more.
+    const int cpb = a.chunk > 0 ? (a.ntiles + a.chunk - 1) / a.chunk : 0;
+    const long long n_chunks = live_blocks * cpb;
+    const int S = gridDim.x;
+    long long reg_g = 0;
+    int reg_n = 0;
+    if (a.chunk <= 0) {
+        const int block = blockIdx.x / a.G, region = blockIdx.x % a.G;
+        const int tile_begin = region * a.tiles_per_region;
+        if (block < live_blocks && tile_begin < a.ntiles) {
+            reg_g = static_cast<long long>(block) * a.ntiles + tile_begin;
+            reg_n = min(a.ntiles, tile_begin + a.tiles_per_region) - tile_begin;
+        }
+    }
+    if (a.chunk > 0 ? n_chunks == 0 : reg_n == 0) {
+        // uniform: no work (no live rotations in the device-driven fallback, or an empty region)
+        if (a.chunk > 0 && threadIdx.x == 0 && atomicAdd(&a.sched[0], 1ull) == static_cast<unsigned>(S - 1))
+            for (int j = 0; j <= S; j++) a.sched[j] = 0;
+        return;
+    }
     unsigned char* rec_smem = smem;   // [main box | pair box at a.rec_stage_bytes]
     unsigned char* w_smem = smem + a.rec_stage_bytes + ((a.box_bytes_pair + 127) & ~127);
 
@@ -428,6 +479,10 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
             dk::mbar_init(&tm_full[i], 1);
             dk::mbar_init(&tm_empty[i], a.nepi);
         }
+        for (int i = 0; i < NCR; i++) {
+            dk::mbar_init(&ch_full[i], 1);
+            dk::mbar_init(&ch_empty[i], 2 + a.nepi);
+        }
         dk::fence_mbar_init();
     }
     if (warp == 1) {
@@ -442,32 +497,108 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
 
     const bool tr = a.trace != nullptr;
     long long tw0 = 0, tw1 = 0, tw2 = 0, tstart = tr ? clock64() : 0;   // per-role trace accumulators
-    if (n_tiles > 0) {
+    const unsigned long long gt0 = tr ? gtimer() : 0;
+    int cs = 0;             // chunk ring slot / phase of this role
+    unsigned cph = 0;
+    // consumer side of the chunk ring (one thread per role; the epilogue warps each arrive once)
+    long long tch = 0;      // chunk-wait cycles of this role (trace)
+    auto take_chunk = [&](long long& g, bool arrive) -> int {
+        twait(&ch_full[cs], cph, tr, tch);
+        g = s_cg[cs];
+        const int n = s_cn[cs];
+        if (arrive) dk::mbar_arrive(&ch_empty[cs]);
+        if (++cs == NCR) {
+            cs = 0;
+            cph ^= 1u;
+        }
+        return n;
+    };
+    int n_tiles = 0;        // tiles this CTA processed (trace)
+    {
         if (warp == 0) {
             // ------------------------------------------------ weight producer (one thread): the whole A
             // stream in stage order; it never waits on a receptor buffer (warp 2 + nepi loads those)
-            if (elect_one()) {
-                const unsigned char* wsrc = a.W + static_cast<size_t>(block) * NSTEPS * WCHUNK;
-                int ws = 0, wph = 0, wuse = 0;
-                for (int ti = 0; ti < n_tiles; ti++) {
-                    for (int s = 0; s < NSTEPS; s += KS) {
-                        if (wuse >= a.wstages) twait(&w_empty[ws], wph ^ 1, tr, tw0);
-                        dk::mbar_arrive_expect_tx(&w_full[ws], STAGE);
-                        dk::bulk_load(w_smem + static_cast<size_t>(ws) * STAGE,
-                                      wsrc + static_cast<size_t>(s) * WCHUNK, STAGE, &w_full[ws]);
-                        wuse++;
-                        if (++ws == a.wstages) {
-                            ws = 0;
-                            wph ^= 1;
+            // (warp-wide: lane 0 streams, all lanes search for chunks to help with)
+            auto seg_lo = [&](int j) -> long long { return static_cast<long long>(j) * n_chunks / S; };
+            int seg = blockIdx.x;
+            auto fetch = [&]() -> long long {   // next chunk id, -1 when every segment is exhausted
+                for (;;) {
+                    long long c = -1;
+                    if (lane == 0) {
+                        const long long t = static_cast<long long>(atomicAdd(&a.sched[1 + seg], 1ull));
+                        if (seg_lo(seg) + t < seg_lo(seg + 1)) c = seg_lo(seg) + t;
+                    }
+                    c = __shfl_sync(0xffffffffu, c, 0);
+                    if (c >= 0) return c;
+                    int found = -1;
+                    for (int base = 1; base < S && found < 0; base += 32) {
+                        bool has = false;
+                        if (base + lane < S) {
+                            const int j = (seg + base + lane) % S;
+                            const unsigned long long t = *reinterpret_cast<volatile unsigned long long*>(&a.sched[1 + j]);
+                            has = seg_lo(j) + static_cast<long long>(t) < seg_lo(j + 1);
+                        }
+                        const unsigned mk = __ballot_sync(0xffffffffu, has);
+                        if (mk) found = (seg + base + __ffs(mk) - 1) % S;
+                    }
+                    if (found < 0) return -1;
+                    seg = found;
+                }
+            };
+            int ws = 0, wph = 0, wuse = 0;
+            long long c = a.chunk > 0 ? fetch() : 0;   // dynamic mode: the chunk to post next
+            for (bool first = true;; first = false) {
+                long long g = 0;
+                int n = 0;
+                if (a.chunk > 0) {
+                    if (c >= 0) {
+                        const long long blk = c / cpb;
+                        const int t0 = static_cast<int>(c % cpb) * a.chunk;
+                        g = blk * a.ntiles + t0;
+                        n = min(a.chunk, a.ntiles - t0);
+                    }
+                } else if (first) {
+                    g = reg_g;
+                    n = reg_n;
+                }
+                // post the chunk (the slot is free once all consumers took the chunk NCR posts ago)
+                if (lane == 0) {
+                    dk::mbar_wait(&ch_empty[cs], cph ^ 1u);
+                    s_cg[cs] = g;
+                    s_cn[cs] = n;
+                    dk::mbar_arrive(&ch_full[cs]);
+                }
+                __syncwarp();
+                if (++cs == NCR) {
+                    cs = 0;
+                    cph ^= 1u;
+                }
+                if (n == 0) break;
+                if (a.chunk > 0) c = fetch();   // one chunk of lookahead: the atomic hides behind the stream
+                n_tiles += n;
+                if (lane == 0) {
+                    const unsigned char* wsrc = a.W + static_cast<size_t>(g / a.ntiles) * NSTEPS * WCHUNK;
+                    for (int ti = 0; ti < n; ti++) {
+                        for (int s = 0; s < NSTEPS; s += KS) {
+                            if (wuse >= a.wstages) twait(&w_empty[ws], wph ^ 1, tr, tw0);
+                            dk::mbar_arrive_expect_tx(&w_full[ws], STAGE);
+                            dk::bulk_load(w_smem + static_cast<size_t>(ws) * STAGE,
+                                          wsrc + static_cast<size_t>(s) * WCHUNK, STAGE, &w_full[ws]);
+                            wuse++;
+                            if (++ws == a.wstages) {
+                                ws = 0;
+                                wph ^= 1;
+                            }
                         }
                     }
                 }
-                if (tr) {
-                    atomicAdd(&a.trace[TR_PROD_TOTAL], static_cast<unsigned long long>(clock64() - tstart));
-                    atomicAdd(&a.trace[TR_PROD_WEMPTY], static_cast<unsigned long long>(tw0));
-                    atomicAdd(&a.trace[TR_CTAS], 1ull);
-                    atomicAdd(&a.trace[TR_TILES], static_cast<unsigned long long>(n_tiles));
-                }
+                __syncwarp();
+            }
+            if (tr && lane == 0) {
+                atomicAdd(&a.trace[TR_PROD_TOTAL], static_cast<unsigned long long>(clock64() - tstart));
+                atomicAdd(&a.trace[TR_PROD_WEMPTY], static_cast<unsigned long long>(tw0));
+                atomicAdd(&a.trace[TR_CTAS], 1ull);
+                atomicAdd(&a.trace[TR_TILES], static_cast<unsigned long long>(n_tiles));
             }
             __syncwarp();
         } else if (warp == 2 + a.nepi) {
@@ -476,23 +607,31 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
             if (elect_one()) {
                 dk::prefetch_tmap(&tmap);
                 dk::prefetch_tmap(&tmap_pair);
-                int tx = tile_begin % a.ntx, ty = (tile_begin / a.ntx) % a.nty, tz = tile_begin / (a.ntx * a.nty);
-                for (int ti = 0; ti < n_tiles; ti++) {
-                    for (int which = 0; which < 2; which++) {
-                        if (ti > 0) twait(&rec_empty[which], (ti - 1) & 1, tr, tw1);
-                        dk::mbar_arrive_expect_tx(&rec_full[which], which ? a.box_bytes_pair : a.box_bytes);
-                        tma_load_5d(rec_smem + which * a.rec_stage_bytes, which ? &tmap_pair : &tmap, 0, tx * NT,
-                                    ty * Q, tz, 0, &rec_full[which]);
-                    }
-                    if (++tx == a.ntx) {
-                        tx = 0;
-                        if (++ty == a.nty) {
-                            ty = 0;
-                            tz++;
+                int ti = 0;   // tiles so far (buffer phases)
+                long long g;
+                for (int n; (n = take_chunk(g, true)) > 0;) {
+                    const int t0 = static_cast<int>(g % a.ntiles);
+                    int tx = t0 % a.ntx, ty = (t0 / a.ntx) % a.nty, tz = t0 / (a.ntx * a.nty);
+                    for (int j = 0; j < n; j++, ti++) {
+                        for (int which = 0; which < 2; which++) {
+                            if (ti > 0) twait(&rec_empty[which], (ti - 1) & 1, tr, tw1);
+                            dk::mbar_arrive_expect_tx(&rec_full[which], which ? a.box_bytes_pair : a.box_bytes);
+                            tma_load_5d(rec_smem + which * a.rec_stage_bytes, which ? &tmap_pair : &tmap, 0,
+                                        tx * NT, ty * Q, tz, 0, &rec_full[which]);
+                        }
+                        if (++tx == a.ntx) {
+                            tx = 0;
+                            if (++ty == a.nty) {
+                                ty = 0;
+                                tz++;
+                            }
                         }
                     }
                 }
-                if (tr) atomicAdd(&a.trace[TR_PROD_REMPTY], static_cast<unsigned long long>(tw1));
+                if (tr) {
+                    atomicAdd(&a.trace[TR_PROD_REMPTY], static_cast<unsigned long long>(tw1));
+                    atomicAdd(&a.trace[TR_REC_CHWAIT], static_cast<unsigned long long>(tch));
+                }
             }
             __syncwarp();
         } else if (warp == 1) {
@@ -531,7 +670,10 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                             wph ^= 1;
                         }
                 };
-                for (int ti = 0; ti < n_tiles; ti++) {
+                int ti = 0;   // tiles so far (buffer phases)
+                long long g;
+                for (int n; (n = take_chunk(g, true)) > 0;)
+                for (int j = 0; j < n; j++, ti++) {
                     twait(&rec_full[0], ti & 1, tr, tw2);
                     tc_fence_after();
                     // pass 1, stages [0, D): row by row, each row after the epilogue released it
@@ -632,6 +774,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                     atomicAdd(&a.trace[TR_MMA_TMEMPTY], static_cast<unsigned long long>(tw0));
                     atomicAdd(&a.trace[TR_MMA_WFULL], static_cast<unsigned long long>(tw1));
                     atomicAdd(&a.trace[TR_MMA_RFULL], static_cast<unsigned long long>(tw2));
+                    atomicAdd(&a.trace[TR_MMA_CHWAIT], static_cast<unsigned long long>(tch));
                 }
             }
             __syncwarp();
@@ -641,39 +784,86 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
             const int cls = (warp - 2) >> 2;
             const int nclass = a.nepi >> 2;
             const int r = quarter * 32 + lane;                  // rotation within the block (TMEM lane)
-            const int slot = block * ROT + r;
-            const bool rot_ok = slot < n_eff;
+            long long cur = -1;                                 // rotation block of the lists
+            int slot = 0;
+            bool rot_ok = false;
             unsigned long long lst[LIST];
 #pragma unroll
             for (int i = 0; i < LIST; i++) lst[i] = KEY_MAX;
             float th = __int_as_float(0x7f800000);   // score of the list's last key (+inf while not full)
             uint32_t th_t = 0xffffffffu;             // t_lin of the list's last key
-            int tx = tile_begin % a.ntx, ty = (tile_begin / a.ntx) % a.nty, tz = tile_begin / (a.ntx * a.nty);
-            for (int ti = 0; ti < n_tiles; ti++) {
-                epi_tile<NT, Q, GRID>(a, tmem, tm_empty, quarter, cls, nclass, lane, slot, rot_ok, tx, ty, tz, lst, th,
-                                      th_t, tr, tw0, tw1, tm_full, ti & 1);
-                if (++tx == a.ntx) {
-                    tx = 0;
-                    if (++ty == a.nty) {
-                        ty = 0;
-                        tz++;
+            int ti = 0;                               // tiles so far (TMEM phases)
+            long long g, tpub = 0;
+            unsigned nins = 0;
+            for (int n; (n = take_chunk(g, false)) > 0;) {
+                __syncwarp();
+                if (lane == 0) dk::mbar_arrive(&ch_empty[(cs + NCR - 1) % NCR]);
+                const long long blk = g / a.ntiles;
+                if (blk != cur) {
+                    // a new rotation block: publish the lists of the previous one (once: the chunk sequence
+                    // of a CTA is increasing, so it never returns to a block)
+                    if constexpr (!GRID) {
+                        const long long tp0 = tr ? clock64() : 0;
+                        if (cur >= 0 && rot_ok) epi_publish(lst, slot, a);
+                        if (tr) tpub += clock64() - tp0;
+                    }
+#pragma unroll
+                    for (int i = 0; i < LIST; i++) lst[i] = KEY_MAX;
+                    th = __int_as_float(0x7f800000);
+                    th_t = 0xffffffffu;
+                    cur = blk;
+                    slot = static_cast<int>(blk) * ROT + r;
+                    rot_ok = slot < n_eff;
+                }
+                const int t0 = static_cast<int>(g % a.ntiles);
+                int tx = t0 % a.ntx, ty = (t0 / a.ntx) % a.nty, tz = t0 / (a.ntx * a.nty);
+                for (int j = 0; j < n; j++, ti++) {
+                    epi_tile<NT, Q, GRID>(a, tmem, tm_empty, quarter, cls, nclass, lane, slot, rot_ok, tx, ty, tz, lst,
+                                          th, th_t, tr, tw0, tw1, tm_full, ti & 1, tr ? &nins : nullptr);
+                    if (++tx == a.ntx) {
+                        tx = 0;
+                        if (++ty == a.nty) {
+                            ty = 0;
+                            tz++;
+                        }
                     }
                 }
             }
+            __syncwarp();
+            if (lane == 0) dk::mbar_arrive(&ch_empty[(cs + NCR - 1) % NCR]);   // the end marker
             if (tr && lane == 0) {
                 atomicAdd(&a.trace[TR_EPI_TOTAL], static_cast<unsigned long long>(clock64() - tstart));
                 atomicAdd(&a.trace[TR_EPI_TMFULL], static_cast<unsigned long long>(tw0));
                 atomicAdd(&a.trace[TR_EPI_LDTM], static_cast<unsigned long long>(tw1));
                 atomicAdd(&a.trace[TR_EPI_WARPS], 1ull);
+                atomicAdd(&a.trace[TR_EPI_CHWAIT], static_cast<unsigned long long>(tch));
+                atomicAdd(&a.trace[TR_EPI_PUB], static_cast<unsigned long long>(tpub));
             }
+            if (tr) atomicAdd(&a.trace[TR_EPI_INS], static_cast<unsigned long long>(nins));
             if constexpr (!GRID) {
-                if (rot_ok) epi_publish(lst, slot, a);
+                if (cur >= 0 && rot_ok) epi_publish(lst, slot, a);
             }
         }
     }
     tc_fence_before();
     __syncthreads();
     if (warp == 1) asm volatile("tcgen05.dealloc.cta_group::1.sync.aligned.b32 %0, 512;" ::"r"(tmem));
+    // dynamic mode: the last CTA to finish (every fetch of every CTA is done by then) resets the counters
+    if (a.chunk > 0 && threadIdx.x == 0 && atomicAdd(&a.sched[0], 1ull) == static_cast<unsigned>(S - 1))
+        for (int j = 0; j <= S; j++) a.sched[j] = 0;
+    if (tr && threadIdx.x == 0) {
+        const unsigned long long gt1 = gtimer();
+        atomicMax(&a.trace[TR_GT_START_NOT], ~gt0);
+        atomicMax(&a.trace[TR_GT_END], gt1);
+        atomicAdd(&a.trace[TR_GT_CTA_NS], gt1 - gt0);
+        if (blockIdx.x < TR_MAXCTA) {
+            unsigned smid;
+            asm volatile("mov.u32 %0, %%smid;" : "=r"(smid));
+            a.trace[TR_CTA0 + 3 * blockIdx.x] = gt0;
+            a.trace[TR_CTA0 + 3 * blockIdx.x + 1] = gt1;
+            a.trace[TR_CTA0 + 3 * blockIdx.x + 2] = smid;
+        }
+    }
 }
 
 // ------------------------------------------------------------------ variant 2: streamed receptor planes

@@ -274,6 +274,46 @@ def test_poses_mid_config(D, orc, kind, rho, engine):
     assert info["fallback_last"] <= 2
 
 
+def test_tc_dynamic_scheduler_across_rotation_blocks(D, orc):
+    """tcgen05 variant 1 runs one persistent CTA per SM that takes 4-tile chunks of (rotation block, tiles)
+    from per-CTA segments of the chunk space and then helps other segments: with 3 blocks of 128 rotations
+    and 370 tiles per block, a CTA's lists change block mid-stream and every block has many publishers.
+    Poses validate against the oracle on units of every block (first / last rotations of each), and the
+    bits equal region mode's (DOCK_TUNE_REGIONS > 0: one CTA per (block, region)), other chunk sizes' and
+    the exact fallback's."""
+    P, m = 4, 4
+    R = g.receptor_ftmap_like((48, 40, 37), P)
+    w = g.weights(P)
+    probes = g.probes(3, m, P)
+    rot = g.rotations(110)
+    n = len(probes) * len(rot)
+    units = sorted({0, 1, 127, 128, 129, 255, 256, 257, n - 1} | set(range(120, 136)))
+    poses, info, _ = _dock_and_validate(D, orc, R, w, probes, rot, 4, 1, units=units, engine=2)
+    assert info["engine_last"] == 2 and info["tc_variant_last"] == 1
+    assert info["regions_last"] == 0 and info["items_last"] <= info["n_sms"]   # dynamic scheduler
+    ctx = _ctx(D, R, w, m, 2)
+
+    def bits(p):
+        return p["rot"], p["t_lin"], p["score"].view(np.uint32)
+
+    for G in (1, 4):
+        D.dock_set_tuning(ctx, D.DOCK_TUNE_REGIONS, G)
+        reg = D.dock_probe_batch(ctx, probes, rot, k=4, rho=1)
+        assert all(np.array_equal(a, b) for a, b in zip(bits(reg), bits(poses)))
+    D.dock_set_tuning(ctx, D.DOCK_TUNE_REGIONS, 0)
+    for chunk in (1, 7, 370, 4096):
+        D.dock_set_tuning(ctx, D.DOCK_TUNE_TC_CHUNK, chunk)
+        for _ in range(2):   # back to back: the scheduler's counters reset themselves between launches
+            dyn = D.dock_probe_batch(ctx, probes, rot, k=4, rho=1)
+            assert all(np.array_equal(a, b) for a, b in zip(bits(dyn), bits(poses))), chunk
+    D.dock_set_tuning(ctx, D.DOCK_TUNE_TC_CHUNK, 0)
+    D.dock_set_tuning(ctx, D.DOCK_TUNE_FORCE_FALLBACK, 1)
+    fb = D.dock_probe_batch(ctx, probes, rot, k=4, rho=1)
+    assert (fb["flags"] & D.DOCK_POSE_FALLBACK).all()
+    assert all(np.array_equal(a, b) for a, b in zip(bits(fb), bits(poses)))
+    ctx.close()
+
+
 @pytest.mark.parametrize("engine", ENGINES)
 @pytest.mark.parametrize("rho,k", [(0, 4), (1, 4), (0, 1)])
 def test_integer_inputs_exact_poses(D, orc, rho, k, engine):
@@ -373,6 +413,17 @@ def test_device_resident_io(D):
     D.dock_probe_batch(ctx, dprobes, torch.from_numpy(rot).cuda(), k=4, rho=1, out=out)
     D.dock_sync(ctx)
     assert np.array_equal(D.poses_from_device(out), host)
+    # a ProbeSet (descriptors marshalled once) over device or host arrays: the same poses, repeatedly
+    for ps in (D.dock_probes(ctx, dprobes), D.dock_probes(ctx, probes)):
+        for _ in range(2):
+            out.fill_(-1)
+            D.dock_probe_batch(ctx, ps, torch.from_numpy(rot).cuda(), k=4, rho=1, out=out)
+            D.dock_sync(ctx)
+            assert np.array_equal(D.poses_from_device(out), host)
+    other = D.dock_init(torch.from_numpy(R[:2]).cuda(), torch.from_numpy(w[:2]).cuda(), H, m_max=m)
+    with pytest.raises(ValueError):
+        D.dock_probe_batch(other, D.dock_probes(ctx, dprobes), rot, k=4, rho=1)
+    other.close()
     ctx.close()
 
 
