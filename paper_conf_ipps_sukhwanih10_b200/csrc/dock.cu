@@ -84,7 +84,7 @@ struct dock_ctx {
     int engine_last = 0;
     int tc_variant = 0;        // DOCK_TUNE_TC_VARIANT: 0 auto, 1 resident boxes (P <= 4), 2 streamed planes
     int tc_chunk = 0;          // DOCK_TUNE_TC_CHUNK: tiles per scheduled chunk (variant 1), 0 = auto
-    unsigned long long* d_sched = nullptr;   // [1 + n_sms] dynamic tile scheduler counters (self-resetting)
+    unsigned long long* d_sched = nullptr;   // [1 + 2 n_sms] dynamic tile scheduler counters (self-resetting)
     int tc_variant_last = 0;
     int tc_m_last = 0;
     int tc_ksteps_last = 0;    // K-steps (of 16) per translation row in the last tcgen05 launch
@@ -1529,10 +1529,10 @@ dock_status dock_init(const dock_grid_desc* g, const float* receptor, const floa
     cudaMemcpy(ctx->d_eye, eye.data(), sizeof(float) * P * P, cudaMemcpyHostToDevice);
     cudaMemcpy(ctx->d_ones, ones.data(), sizeof(float) * P, cudaMemcpyHostToDevice);
     cudaMemsetAsync(ctx->d_small, 0, 64, ctx->stream);
-    // tcgen05 dynamic tile scheduler: [CTAs done, chunks taken per segment (one per CTA <= n_sms)], zero
+    // tcgen05 dynamic tile scheduler: [CTAs done, chunks taken per segment (< 2 n_sms segments)], zero
     // between launches (the last CTA of each launch resets it); without it variant 1 runs region mode
-    if (cudaMalloc(&ctx->d_sched, sizeof(unsigned long long) * (ctx->n_sms + 2)) == cudaSuccess)
-        cudaMemsetAsync(ctx->d_sched, 0, sizeof(unsigned long long) * (ctx->n_sms + 2), ctx->stream);
+    if (cudaMalloc(&ctx->d_sched, sizeof(unsigned long long) * (2 * ctx->n_sms + 2)) == cudaSuccess)
+        cudaMemsetAsync(ctx->d_sched, 0, sizeof(unsigned long long) * (2 * ctx->n_sms + 2), ctx->stream);
     else
         ctx->d_sched = nullptr;
     cudaGetLastError();
@@ -1849,7 +1849,8 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
                     "\"epi_ldtm\": %.0f, \"prod_total\": %.0f, \"prod_wait_w_empty\": %.0f, "
                     "\"prod_wait_rec_empty\": %.0f, \"span_ms\": %.4f, \"cta_ms\": %.4f, "
                     "\"epi_wait_chunk\": %.0f, \"mma_wait_chunk\": %.0f, \"rec_wait_chunk\": %.0f, "
-                    "\"epi_publish\": %.0f, \"inserts_per_tile_lane\": %.3f}\n",
+                    "\"epi_publish\": %.0f, \"inserts_per_tile_lane\": %.3f, \"gates_per_tile_lane\": %.3f, "
+                    "\"rare_entries_per_tile_warp\": %.3f}\n",
                     v, h[tc::TR_CTAS], h[tc::TR_TILES] / c, h[tc::TR_MMA_TOTAL] / c,
                     h[tc::TR_MMA_TMEMPTY] / c, h[tc::TR_MMA_WFULL] / c, h[tc::TR_MMA_RFULL] / c,
                     h[tc::TR_EPI_TOTAL] / e, h[tc::TR_EPI_TMFULL] / e, h[tc::TR_EPI_LDTM] / e,
@@ -1857,7 +1858,9 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
                     h[tc::TR_GT_END] ? (h[tc::TR_GT_END] - ~h[tc::TR_GT_START_NOT]) * 1e-6 : 0.0,
                     h[tc::TR_GT_CTA_NS] * 1e-6 / c, h[tc::TR_EPI_CHWAIT] / e, h[tc::TR_MMA_CHWAIT] / c,
                     h[tc::TR_REC_CHWAIT] / c, h[tc::TR_EPI_PUB] / e,
-                    h[tc::TR_TILES] ? h[tc::TR_EPI_INS] / (double(h[tc::TR_TILES]) * tc::ROT) : 0.0);
+                    h[tc::TR_TILES] ? h[tc::TR_EPI_INS] / (double(h[tc::TR_TILES]) * tc::ROT) : 0.0,
+                    h[tc::TR_TILES] ? h[tc::TR_EPI_GATE] / (double(h[tc::TR_TILES]) * tc::ROT) : 0.0,
+                    h[tc::TR_TILES] ? h[tc::TR_EPI_WRARE] / (double(h[tc::TR_TILES]) * ta.nepi) : 0.0);
         }
         ctx->regions_last = ta.chunk > 0 ? 0 : G;
         ctx->items_last = items;

@@ -90,7 +90,9 @@ enum { TR_CTAS = 0, TR_TILES, TR_MMA_TOTAL, TR_MMA_TMEMPTY, TR_MMA_WFULL, TR_MMA
        TR_MMA_CHWAIT = 17,
        TR_REC_CHWAIT = 18,
        TR_EPI_PUB = 19,        // epilogue: publishing lists (cycles)
-       TR_EPI_INS = 20,        // epilogue: list insertions (all lanes)
+       TR_EPI_INS = 20,        // epilogue: list insertions, lane gate passes, warp rare-path entries
+       TR_EPI_GATE = 21,
+       TR_EPI_WRARE = 22,
        TR_CTA0 = 24,           // per CTA (blockIdx.x < TR_MAXCTA): start, end (globaltimer), SM id
        TR_MAXCTA = 1024,
        TR_N = TR_CTA0 + 3 * TR_MAXCTA };
@@ -242,7 +244,12 @@ __device__ __forceinline__ void epi_chunk(const uint32_t (&v)[32], unsigned long
         for (int j = 1; j < 32; j++) mn = fminf(mn, __uint_as_float(v[j]));
         // exact gate: a strictly better score, or a tie that could carry a smaller t_lin (exact-zero
         // scores in empty space tie constantly)
-        if (mn < th || (mn == th && tbase + c0 < th_t)) {
+        const bool gate = mn < th || (mn == th && tbase + c0 < th_t);
+        if (nins) {   // trace: [0] insertions, [1] lane gate passes, [2] warp entries into the rare path
+            nins[1] += gate;
+            nins[2] += __any_sync(__activemask(), gate) ? 1u : 0u;
+        }
+        if (gate) {
             // rare path: bitmask of candidates, each extracted with a 5-level select tree (no local memory)
             uint32_t msk = 0;
 #pragma unroll
@@ -254,7 +261,7 @@ __device__ __forceinline__ void epi_chunk(const uint32_t (&v)[32], unsigned long
                 if (sv <= th) {
                     const unsigned long long key = dk::make_key(sv, tbase + c0 + j);
                     if (key < lst[LIST - 1]) {
-                        if (nins) ++*nins;
+                        if (nins) ++nins[0];
                         list_insert(lst, key);
                         th = dk::key_score_bound(static_cast<uint32_t>(lst[LIST - 1] >> 32));
                         th_t = static_cast<uint32_t>(lst[LIST - 1] & 0xffffffffu);
@@ -439,14 +446,19 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
     const long long live_blocks = (n_eff + ROT - 1) / ROT;
     // Work: a sequence of chunks (g, n) = n consecutive tiles of one rotation block starting at the (block,
     // tile) pair g = block * ntiles + tile.  Region mode: the one chunk (block, region) of this CTA.  Dynamic
-    // mode: chunk c = (block c / cpb, tiles [(c % cpb) chunk, ..)), c in [0, n_chunks) split into S =
-    // gridDim.x contiguous segments with one counter each.  A CTA takes the chunks of its own segment in
-    // order (a contiguous range, so its top-k lists live long: a list restart costs a burst of insertions),
+    // mode: chunk c = (block c / cpb, tiles [(c % cpb) chunk, ..)), c in [0, n_chunks), split into NS
+    // segments with one counter each.  A CTA takes the chunks of its own segment in order (a contiguous
+    // tile range of one block, so its top-k lists live long: a list restart costs a burst of insertions),
     // then helps the next segments that still have chunks: CTAs whose tiles are cheaper (per-tile cost
-    // varies with the receptor region through the epilogue's insertions) take more.
+    // varies with the receptor region through the epilogue's insertions) take more.  The NS = S =
+    // gridDim.x segments are contiguous ranges of the chunk space, so concurrent CTAs read the receptor at
+    // scattered positions: that costs L2 misses (~2.2 GB of DRAM reads per prod launch instead of ~0.1)
+    // but spreads the reads over the L2 slices; region-major segments that keep the CTAs in step on a few
+    // receptor windows cut DRAM to 0.1 GB and ran 13 % slower (hot L2 lines).
     const int cpb = a.chunk > 0 ? (a.ntiles + a.chunk - 1) / a.chunk : 0;
     const long long n_chunks = live_blocks * cpb;
     const int S = gridDim.x;
+    const int NS = S;
     long long reg_g = 0;
     int reg_n = 0;
     if (a.chunk <= 0) {
@@ -460,7 +472,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
     if (a.chunk > 0 ? n_chunks == 0 : reg_n == 0) {
         // uniform: no work (no live rotations in the device-driven fallback, or an empty region)
         if (a.chunk > 0 && threadIdx.x == 0 && atomicAdd(&a.sched[0], 1ull) == static_cast<unsigned>(S - 1))
-            for (int j = 0; j <= S; j++) a.sched[j] = 0;
+            for (int j = 0; j <= NS; j++) a.sched[j] = 0;
         return;
     }
     unsigned char* rec_smem = smem;   // [main box | pair box at a.rec_stage_bytes]
@@ -519,27 +531,35 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
             // ------------------------------------------------ weight producer (one thread): the whole A
             // stream in stage order; it never waits on a receptor buffer (warp 2 + nepi loads those)
             // (warp-wide: lane 0 streams, all lanes search for chunks to help with)
-            auto seg_lo = [&](int j) -> long long { return static_cast<long long>(j) * n_chunks / S; };
+            // segment j: chunk ids [lo, hi)
+            auto seg_range = [&](int j, long long& lo, long long& hi) {
+                lo = static_cast<long long>(j) * n_chunks / NS;
+                hi = static_cast<long long>(j + 1) * n_chunks / NS;
+            };
             int seg = blockIdx.x;
             auto fetch = [&]() -> long long {   // next chunk id, -1 when every segment is exhausted
                 for (;;) {
                     long long c = -1;
                     if (lane == 0) {
+                        long long lo, hi;
+                        seg_range(seg, lo, hi);
                         const long long t = static_cast<long long>(atomicAdd(&a.sched[1 + seg], 1ull));
-                        if (seg_lo(seg) + t < seg_lo(seg + 1)) c = seg_lo(seg) + t;
+                        if (lo + t < hi) c = lo + t;
                     }
                     c = __shfl_sync(0xffffffffu, c, 0);
                     if (c >= 0) return c;
                     int found = -1;
-                    for (int base = 1; base < S && found < 0; base += 32) {
+                    for (int base = 1; base < NS && found < 0; base += 32) {
                         bool has = false;
-                        if (base + lane < S) {
-                            const int j = (seg + base + lane) % S;
+                        if (base + lane < NS) {
+                            const int j = (seg + base + lane) % NS;
+                            long long lo, hi;
+                            seg_range(j, lo, hi);
                             const unsigned long long t = *reinterpret_cast<volatile unsigned long long*>(&a.sched[1 + j]);
-                            has = seg_lo(j) + static_cast<long long>(t) < seg_lo(j + 1);
+                            has = lo + static_cast<long long>(t) < hi;
                         }
                         const unsigned mk = __ballot_sync(0xffffffffu, has);
-                        if (mk) found = (seg + base + __ffs(mk) - 1) % S;
+                        if (mk) found = (seg + base + __ffs(mk) - 1) % NS;
                     }
                     if (found < 0) return -1;
                     seg = found;
@@ -794,7 +814,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
             uint32_t th_t = 0xffffffffu;             // t_lin of the list's last key
             int ti = 0;                               // tiles so far (TMEM phases)
             long long g, tpub = 0;
-            unsigned nins = 0;
+            unsigned nins[3] = {0, 0, 0};
             for (int n; (n = take_chunk(g, false)) > 0;) {
                 __syncwarp();
                 if (lane == 0) dk::mbar_arrive(&ch_empty[(cs + NCR - 1) % NCR]);
@@ -819,7 +839,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                 int tx = t0 % a.ntx, ty = (t0 / a.ntx) % a.nty, tz = t0 / (a.ntx * a.nty);
                 for (int j = 0; j < n; j++, ti++) {
                     epi_tile<NT, Q, GRID>(a, tmem, tm_empty, quarter, cls, nclass, lane, slot, rot_ok, tx, ty, tz, lst,
-                                          th, th_t, tr, tw0, tw1, tm_full, ti & 1, tr ? &nins : nullptr);
+                                          th, th_t, tr, tw0, tw1, tm_full, ti & 1, tr ? nins : nullptr);
                     if (++tx == a.ntx) {
                         tx = 0;
                         if (++ty == a.nty) {
@@ -839,7 +859,11 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                 atomicAdd(&a.trace[TR_EPI_CHWAIT], static_cast<unsigned long long>(tch));
                 atomicAdd(&a.trace[TR_EPI_PUB], static_cast<unsigned long long>(tpub));
             }
-            if (tr) atomicAdd(&a.trace[TR_EPI_INS], static_cast<unsigned long long>(nins));
+            if (tr) {
+                atomicAdd(&a.trace[TR_EPI_INS], static_cast<unsigned long long>(nins[0]));
+                atomicAdd(&a.trace[TR_EPI_GATE], static_cast<unsigned long long>(nins[1]));
+                if (lane == 0) atomicAdd(&a.trace[TR_EPI_WRARE], static_cast<unsigned long long>(nins[2]));
+            }
             if constexpr (!GRID) {
                 if (cur >= 0 && rot_ok) epi_publish(lst, slot, a);
             }
@@ -850,7 +874,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
     if (warp == 1) asm volatile("tcgen05.dealloc.cta_group::1.sync.aligned.b32 %0, 512;" ::"r"(tmem));
     // dynamic mode: the last CTA to finish (every fetch of every CTA is done by then) resets the counters
     if (a.chunk > 0 && threadIdx.x == 0 && atomicAdd(&a.sched[0], 1ull) == static_cast<unsigned>(S - 1))
-        for (int j = 0; j <= S; j++) a.sched[j] = 0;
+        for (int j = 0; j <= NS; j++) a.sched[j] = 0;
     if (tr && threadIdx.x == 0) {
         const unsigned long long gt1 = gtimer();
         atomicMax(&a.trace[TR_GT_START_NOT], ~gt0);

@@ -30,6 +30,7 @@ def main():
               for p in g.probes(c.n_probes, c.m, c.P)]
     rot = torch.from_numpy(g.rotations(c.n_rot)).to(dev)
     ctx = D.dock_init(torch.from_numpy(R).to(dev), torch.from_numpy(w).to(dev), g.SPACING, m_max=c.m, device=0)
+    probes = D.dock_probes(ctx, probes)   # descriptors marshalled once, as bench.py does
     D.dock_set_tuning(ctx, D.DOCK_TUNE_ENGINE, {"auto": 0, "ffma": 1, "tc": 2, "sparse": 4}[args.engine])
     n = c.n_probes * c.n_rot
     out = torch.empty((n, c.k, 4), dtype=torch.int32, device=dev)

@@ -16,5 +16,6 @@ echo "== launch list prod"
 timeout 900 ncu --metrics gpu__time_duration.sum --clock-control none --csv --log-file gpurun_out/launches_${TAG}_prod.csv \
     python bench.py --steps 2 --warmup 1 --no-e2e --no-cpu-baseline --no-alt > gpurun_out/launches_${TAG}_prod.log 2>&1; echo "rc=$?"
 echo "== full capture k_corr_tc (prod)"; SKIP=1 bash scripts/ncu_kernel.sh ${TAG}_prod_tc k_corr_tc --config prod --engine tc
-echo "== full capture k_corr_sparse (large, 512 rotations)"; SKIP=1 bash scripts/ncu_kernel.sh ${TAG}_large_sparse k_corr_sparse --config large --rotations 512 --engine sparse
+echo "== full capture k_corr_sparse (c64 bench launch)"; SKIP=1 bash scripts/ncu_kernel.sh ${TAG}_c64_sparse k_corr_sparse --config c64
+echo "== full capture k_corr_sparse (large shard bench launch, 8750 rotations)"; SKIP=1 bash scripts/ncu_kernel.sh ${TAG}_large_sparse k_corr_sparse --config large --rotations 8750
 ls gpurun_out | head -50

@@ -35,6 +35,7 @@ def main():
               for p in g.probes(c.n_probes, c.m, c.P)]
     rot = torch.from_numpy(g.rotations(c.n_rot)).to(dev)
     ctx = D.dock_init(torch.from_numpy(R).to(dev), torch.from_numpy(w).to(dev), g.SPACING, m_max=c.m, device=0)
+    probes = D.dock_probes(ctx, probes)   # descriptors marshalled once, as bench.py does
     n = c.n_probes * c.n_rot
     flush = torch.empty(64 << 20, dtype=torch.float32, device=dev)
     res = {"config": args.config, "units": n, "note": __doc__.split("\n")[1].strip(), "per_n": {}}
