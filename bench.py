@@ -57,6 +57,8 @@ def parse():
     ap.add_argument("--no-alt", action="store_true", help="skip the secondary measurement of the other engine")
     ap.add_argument("--tc-epi", type=int, default=0, choices=[0, 4, 8, 16], help="tcgen05 epilogue warps (0 auto)")
     ap.add_argument("--tc-chunk", type=int, default=0, help="tcgen05 tiles per scheduled chunk (0 auto)")
+    ap.add_argument("--tc-schedule", type=int, default=0, choices=[0, 1, 2],
+                    help="tcgen05 variant-1 K-step schedule: 0 occupancy + clustering, 1 occupancy, 2 dense")
     ap.add_argument("--tc-variant", type=int, default=0, choices=[0, 1, 2],
                     help="tcgen05 kernel: 0 auto, 1 = resident receptor boxes (P <= 4), 2 = streamed (group, z-plane) units")
     return ap.parse_args()
@@ -249,7 +251,11 @@ def roofline(pk, pk_kind, info, c, flops_launch, corr_ms, ms_step, units_local):
                 "launch_ms": corr_ms, "kernel_share_of_step": corr_ms / ms_step if ms_step > 0 else None}
     if info["engine_last"] == 2:
         peak = float(pk.get("bf16_tflops", 1590.0))
-        ks = int(info.get("tc_ksteps_last", 0)) or 2 * c.m * c.m * ((c.m + 1) // 2)
+        ks_dense = int(info.get("tc_ksteps_last", 0)) or 2 * c.m * c.m * ((c.m + 1) // 2)
+        ks_exec = float(info.get("tc_ksteps_exec_last", -1.0))
+        # variant 1 runs each rotation block's occupied K-steps only (occupancy schedule): the executed count
+        # is the launch's average over its blocks
+        ks = ks_exec if ks_exec > 0 else ks_dense
         # executed bf16 MMA FLOPs: K = 16 per step, ks steps per translation row (bf16x3 split + padding),
         # times the x / y tiling waste of the launch's row width and rows per tile
         ntt, q = int(info.get("tc_row_last", 128)) or 128, int(info.get("tc_rows_per_tile_last", 4)) or 4
@@ -266,6 +272,7 @@ def roofline(pk, pk_kind, info, c, flops_launch, corr_ms, ms_step, units_local):
                 # the measured cuBLAS figure was taken under the power cap; mostly-zero probe weights draw
                 # less power and keep this kernel at max SM clock, so it is also quoted against the nominal
                 "executed_frac_of_nominal_2250": executed / (corr_ms / 1000.0) / 1e12 / 2250.0,
+                "ksteps_per_row_executed": ks, "ksteps_per_row_dense": ks_dense,
                 "fp32_equiv_frac": achieved / (n_sms * 128 * 2 * float(pk.get("sm_max_mhz", 1965.0)) * 1e6 / 1e12),
                 "flops_per_launch": flops_launch, "launch_ms": corr_ms,
                 "kernel_share_of_step": corr_ms / ms_step if ms_step > 0 else None}
@@ -305,6 +312,7 @@ def run_ours(args):
     D.dock_set_tuning(ctx, D.DOCK_TUNE_TC_VARIANT, args.tc_variant)
     D.dock_set_tuning(ctx, 6, args.tc_epi)   # DOCK_TUNE_TC_EPILOGUE_WARPS
     D.dock_set_tuning(ctx, D.DOCK_TUNE_TC_CHUNK, args.tc_chunk)
+    D.dock_set_tuning(ctx, D.DOCK_TUNE_TC_SCHEDULE, args.tc_schedule)
     probes_dev = [{"xyz": torch.from_numpy(p.xyz).to(dev), "coef": torch.from_numpy(p.coef).to(dev), "m": p.m}
                   for p in probes]
     # probe descriptors marshalled once (the probe arrays stay where they are: device here, host in e2e)

@@ -177,8 +177,16 @@ typedef enum {
                                      other one. */
     DOCK_TUNE_TC_EPILOGUE_WARPS = 6, /* tcgen05 epilogue warps: 0 auto (= the compiled maximum, 8), 4 or 8 (values
                                      above the compiled maximum are clamped to it) */
-    DOCK_TUNE_TC_CHUNK = 7        /* tcgen05 variant 1: tiles per dynamically scheduled chunk (0 = auto, 4;
+    DOCK_TUNE_TC_CHUNK = 7,       /* tcgen05 variant 1: tiles per dynamically scheduled chunk (0 = auto, 4;
                                      1..4096); one persistent CTA per SM takes chunks from a device counter */
+    DOCK_TUNE_TC_SCHEDULE = 8     /* tcgen05 variant 1 K-step schedule.  A K-step (16 products per accumulator) whose
+                                     probe weights are zero for all 128 rotations of a block adds exact zeros, so a
+                                     block runs only its occupied K-steps (a probe grid has at most one occupied voxel
+                                     per atom).  0 (default): occupancy schedule, and for m <= 4 the
+                                     units are first grouped into blocks with few distinct occupied K-steps (greedy,
+                                     on the device); 1: occupancy schedule over blocks of consecutive units; 2: dense
+                                     (every K-step).  Scores are bitwise identical in all three modes (skipped
+                                     products are exact zeros). */
 } dock_tune_key;
 
 dock_status dock_set_tuning(dock_ctx* ctx, int key, int64_t value);
@@ -209,6 +217,8 @@ typedef struct {
     int sp_row_last;           /* sparse engine: translations per column row (32 x per-lane count) */
     double sp_terms_last;      /* sparse engine: atoms summed over the units of the last call (gathers per translation) */
     int sp_zt_last;            /* sparse engine: z planes per warp and step of the last call (1 or 2) */
+    double tc_ksteps_exec_last; /* tcgen05 variant 1: K-steps per translation row executed by the last call, averaged
+                                  over its rotation blocks (occupancy schedule); -1 if none or not yet synced */
 } dock_info;
 
 dock_status dock_get_info(const dock_ctx* ctx, dock_info* info);

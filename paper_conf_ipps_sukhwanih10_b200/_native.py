@@ -25,6 +25,7 @@ DOCK_TUNE_ENGINE = 4
 DOCK_TUNE_TC_VARIANT = 5
 DOCK_TUNE_TC_EPILOGUE_WARPS = 6
 DOCK_TUNE_TC_CHUNK = 7
+DOCK_TUNE_TC_SCHEDULE = 8
 DOCK_ENGINE_AUTO, DOCK_ENGINE_FFMA, DOCK_ENGINE_TC, DOCK_ENGINE_FFT, DOCK_ENGINE_SPARSE = 0, 1, 2, 3, 4
 
 STATUS_NAMES = {0: "DOCK_OK", -1: "DOCK_E_INVALID_ARG", -2: "DOCK_E_UNSUPPORTED",
@@ -56,7 +57,8 @@ class dock_info(C.Structure):
                 ("tc_variant_last", C.c_int), ("tc_ksteps_last", C.c_int),
                 ("tc_row_last", C.c_int), ("tc_rows_per_tile_last", C.c_int), ("pending", C.c_int),
                 ("fb_chunk", C.c_int), ("sp_atom_grids_last", C.c_int), ("sp_row_last", C.c_int),
-                ("sp_terms_last", C.c_double), ("sp_zt_last", C.c_int)]
+                ("sp_terms_last", C.c_double), ("sp_zt_last", C.c_int),
+                ("tc_ksteps_exec_last", C.c_double)]
 
 
 EXPORTS = ["dock_init", "dock_probe", "dock_probe_batch", "dock_sync", "dock_score_grid", "dock_voxelize",

@@ -89,18 +89,26 @@ struct dock_ctx {
     int tc_m_last = 0;
     int tc_ksteps_last = 0;    // K-steps (of 16) per translation row in the last tcgen05 launch
     int tc_nepi = 0;           // epilogue warps (0 = tc::NEPI_MAX)
+    int tc_sched = 0;          // DOCK_TUNE_TC_SCHEDULE: 0 occupancy tables + clustering (m <= 4), 1 occupancy
+                               // tables over consecutive units, 2 dense (every K-step)
+    int tc_blocks_last = 0;
+    bool tc_perm_on = false;   // the main pass's variant-1 blocks use the clustering permutation    // rotation blocks of the last variant-1 launch (executed K-step statistics)
     uint16_t* d_rec_tc = nullptr;     // [g][Zp][Yp][Xp][8] bf16 (hi_0..3, lo_0..3)
     uint16_t* d_rec_pair = nullptr;   // [g][Zp][Yp][Xp][8] bf16 (hi_0..3(X), hi_0..3(X+1))
     int tc_Gch = 0, tc_Xp = 0, tc_Yp = 0, tc_Zp = 0;
     int tcs_ntt = 128;         // variant 2 translations per MMA row, chosen for nx
     TcPlan tcplan[3][DOCK_MAX_M + 1];   // [variant][m]
     DevBuf Wtc;
+    // variant 1 occupancy schedule of the main pass / of the fallback: K-step tables, source steps, per-block
+    // (stages, first pair entry), clustering permutation and unit masks
+    DevBuf tc_ksrc, tc_kinfo, tc_perm, tc_umask, fb_ksrc, fb_kinfo;
     // diagnostics (environment, read at init): DOCK_TC_TRACE=1 prints per-role cycle counters of every
     // tcgen05 launch to stderr
     unsigned long long* d_trace = nullptr;
     // per-call scratch (grow-only)
     DevBuf xyz, coef, off, rot, Lw, T, mu, cnt, cand, poses, fb_list, grid, slots, units, Lw_fb, picks;
-    int* d_small = nullptr;    // [0] status bits (sticky until the next sync point), [1] fb_cnt, [2] cand_max
+    int* d_small = nullptr;    // [0] status bits (sticky until the next sync point), [1] fb_cnt, [2] cand_max,
+                               // [3] K-steps per tile summed over the blocks of the last variant-1 launch
     int* h_small = nullptr;    // pinned mirror, written by the async copy at the end of every call
     void* h_stage = nullptr;   // pinned scratch of the synchronous FFT comparison engine
     size_t h_stage_cap = 0;
@@ -660,6 +668,11 @@ tc::TcArgs tc_args(dock_ctx* ctx, int m, int v, int n_slots, int G, const unsign
     a.tiles_per_region = (a.ntiles + G - 1) / G;
     a.nsteps = tp.nsteps;
     a.W = W;
+    if (v == 1) {   // main pass tables unless W is the fallback's operand
+        const bool fb = W == static_cast<const unsigned char*>(ctx->fb_W.p);
+        a.kinfo = static_cast<const int4*>(fb ? ctx->fb_kinfo.p : ctx->tc_kinfo.p);
+        a.perm = (!fb && ctx->tc_perm_on) ? static_cast<const int*>(ctx->tc_perm.p) : nullptr;
+    }
     a.box_bytes = tp.box_bytes;
     a.box_bytes_pair = tp.box_bytes_pair;
     a.rec_stage_bytes = tp.rec_stage_bytes;
@@ -967,21 +980,52 @@ sp::SpArgs sp_args(dock_ctx* ctx, const SpCall& sc, const sp::Group* d_groups, i
     return a;
 }
 
-// Pack folded FP32 weights into the tcgen05 A-operand layout of variant v.
-dock_status pack_weights_tc(dock_ctx* ctx, int m, int v, int n_slots, const float* Lw, DevBuf* dst = nullptr)
+// Pack folded FP32 weights into the tcgen05 A-operand layout of variant v.  Variant 1 first builds the
+// occupancy schedule (dock_tc.cuh): unit K-step masks and the greedy block clustering (main pass, m <= 4,
+// DOCK_TUNE_TC_SCHEDULE 0), then per block the table of occupied K-steps, then the A operand in table order.
+// fb: the fallback's buffers (no clustering; n_live = the live count of the device-driven loop).
+dock_status pack_weights_tc(dock_ctx* ctx, int m, int v, int n_slots, const float* Lw, bool fb = false,
+                            const unsigned* n_live = nullptr)
 {
     const TcPlan& tp = ctx->tcplan[v][m];
     const int64_t n_blocks = (n_slots + tc::ROT - 1) / tc::ROT;
-    DevBuf& Wb = dst ? *dst : ctx->Wtc;
+    DevBuf& Wb = fb ? ctx->fb_W : ctx->Wtc;
     TRY(ensure(ctx, Wb, (size_t)n_blocks * tp.nsteps * tc::WCHUNK));
     const int64_t rows = n_blocks * tp.nsteps * 2 * tc::ROT;
     const int grid = (int)std::min<int64_t>((rows + 255) / 256, 65535);
     unsigned char* W = static_cast<unsigned char*>(Wb.p);
-    if (v == 1)
-        tc::k_pack_weights_tc_pair<<<grid, 256, 0, ctx->stream>>>(Lw, W, n_slots, ctx->P, m, tp.S1, tp.S1p, tp.S2,
-                                                                   tp.S2p);
-    else
+    if (v == 1) {
+        DevBuf& ks = fb ? ctx->fb_ksrc : ctx->tc_ksrc;
+        DevBuf& ki = fb ? ctx->fb_kinfo : ctx->tc_kinfo;
+        TRY(ensure(ctx, ks, sizeof(uint16_t) * n_blocks * tp.nsteps));
+        TRY(ensure(ctx, ki, sizeof(int4) * n_blocks));
+        const int* perm = nullptr;
+        if (!fb && ctx->tc_sched == 0 && tp.nsteps <= 64 * tc::KSTEPS && n_slots > tc::ROT) {
+            TRY(ensure(ctx, ctx->tc_umask, sizeof(unsigned long long) * n_slots));
+            TRY(ensure(ctx, ctx->tc_perm, sizeof(int) * n_blocks * tc::ROT));
+            auto* um = static_cast<unsigned long long*>(ctx->tc_umask.p);
+            tc::k_tc_unit_masks<<<(n_slots + 127) / 128, 128, 0, ctx->stream>>>(Lw, n_slots, ctx->P, m, um);
+            CU(cudaGetLastError());
+            tc::k_tc_cluster<<<(n_slots + tc::CL_W - 1) / tc::CL_W, tc::CL_THREADS, 0, ctx->stream>>>(
+                um, n_slots, static_cast<int*>(ctx->tc_perm.p));
+            CU(cudaGetLastError());
+            ctx->kernels_last += 2;
+            perm = static_cast<const int*>(ctx->tc_perm.p);
+        }
+        ctx->tc_perm_on = perm != nullptr;
+        tc::k_tc_block_tables<<<(int)n_blocks, 128, 0, ctx->stream>>>(
+            Lw, perm, n_slots, n_live, ctx->P, m, tp.nsteps, (ctx->tc_sched == 2 || tp.nsteps > 64 * tc::KSTEPS) ? 1 : 0,
+            static_cast<uint16_t*>(ks.p), static_cast<int4*>(ki.p),
+            fb ? nullptr : reinterpret_cast<unsigned*>(ctx->d_small + 3));
+        CU(cudaGetLastError());
+        tc::k_pack_weights_tc1<<<grid, 256, 0, ctx->stream>>>(Lw, perm, static_cast<const uint16_t*>(ks.p),
+                                                               static_cast<const int4*>(ki.p), W, n_slots, ctx->P,
+                                                               m, tp.nsteps);
+        ctx->kernels_last++;
+        if (!fb) ctx->tc_blocks_last = (int)n_blocks;
+    } else {
         tc::k_pack_weights_tcs<<<grid, 256, 0, ctx->stream>>>(Lw, W, n_slots, ctx->P, m, tp.nsteps);
+    }
     CU(cudaGetLastError());
     ctx->kernels_last++;
     return DOCK_OK;
@@ -1076,7 +1120,7 @@ dock_status run_grid_tc(dock_ctx* ctx, int m, int n_slots, const float* Lw, floa
 struct FbKey {   // everything the captured fallback graph bakes in (compared bytewise)
     int m, kind, v, G, k, rho, ch, nepi, P, nx, ny, nz;
     int sp_nat, sp_npl, sp_smem, sp_xts;
-    const void *fb_list, *d_small, *dyn, *grid, *Lw, *W, *picks, *slots, *ctl, *w;
+    const void *fb_list, *d_small, *dyn, *grid, *Lw, *W, *picks, *slots, *ctl, *w, *ksrc, *kinfo;
     const void *spG, *sp_tv, *sp_ts, *sp_nt, *sp_dw, *sp_sa, *fb_groups;
 };
 static_assert(sizeof(FbKey) <= sizeof(((dock_ctx*)nullptr)->fb_key), "fb_key too small");
@@ -1138,7 +1182,7 @@ dock_status enqueue_fb_body(dock_ctx* ctx, const FbKey& key, const dk::FbDyn* d_
             dk::k_voxelize_dyn<<<(nvox + 127) / 128, 128, 0, st>>>(&d_dyn->vox);
             CU(cudaGetLastError());
             if (key.kind == ENG_TC) {
-                TRY(pack_weights_tc(ctx, m, key.v, ch, Lw, &ctx->fb_W));
+                TRY(pack_weights_tc(ctx, m, key.v, ch, Lw, true, &ctl->n_live));
                 tc::TcArgs a = tc_args(ctx, m, key.v, ch, key.G, static_cast<const unsigned char*>(ctx->fb_W.p));
                 a.grid = grid;
                 a.n_live = &ctl->n_live;
@@ -1268,6 +1312,8 @@ dock_status launch_fallback(dock_ctx* ctx, int m, int kind, int k, int rho, cons
         key.G = G;
         const TcPlan& tp = ctx->tcplan[vv][m];
         TRY(ensure(ctx, ctx->fb_W, (size_t)tp.nsteps * tc::WCHUNK));
+        TRY(ensure(ctx, ctx->fb_ksrc, sizeof(uint16_t) * tp.nsteps));
+        TRY(ensure(ctx, ctx->fb_kinfo, sizeof(int4)));
     } else if (kind == ENG_FFMA) {
         key.G = choose_regions(ctx, (ch + dk::RB - 1) / dk::RB);
     }
@@ -1285,6 +1331,8 @@ dock_status launch_fallback(dock_ctx* ctx, int m, int kind, int k, int rho, cons
     key.grid = ctx->fb_grid.p;
     key.Lw = ctx->fb_Lw.p;
     key.W = ctx->fb_W.p;
+    key.ksrc = ctx->fb_ksrc.p;
+    key.kinfo = ctx->fb_kinfo.p;
     key.picks = ctx->fb_picks.p;
     key.slots = ctx->fb_slots.p;
     key.ctl = ctx->fb_ctl.p;
@@ -1394,7 +1442,8 @@ void dock_destroy(dock_ctx* ctx)
     DevBuf* bufs[] = {&ctx->xyz,     &ctx->coef,     &ctx->off,    &ctx->rot,      &ctx->Lw,       &ctx->T,
                       &ctx->mu,      &ctx->cnt,      &ctx->cand,   &ctx->poses,    &ctx->fb_list,  &ctx->grid,
                       &ctx->slots,   &ctx->units,    &ctx->Lw_fb,  &ctx->picks,    &ctx->fb_grid,  &ctx->fb_Lw,
-                      &ctx->fb_W,    &ctx->fb_picks, &ctx->fb_slots, &ctx->fb_ctl};
+                      &ctx->fb_W,    &ctx->fb_picks, &ctx->fb_slots, &ctx->fb_ctl,   &ctx->tc_ksrc,
+                      &ctx->tc_kinfo, &ctx->tc_perm, &ctx->tc_umask, &ctx->fb_ksrc, &ctx->fb_kinfo};
     for (DevBuf* b : bufs)
         if (b->p) cudaFree(b->p);
     if (ctx->d_trace) cudaFree(ctx->d_trace);
@@ -1620,6 +1669,10 @@ dock_status dock_set_tuning(dock_ctx* ctx, int key, int64_t value)
             if (value < 0 || value > 4096) return fail(ctx, DOCK_E_INVALID_ARG, "tc chunk must be 0..4096");
             ctx->tc_chunk = (int)value;
             return DOCK_OK;
+        case DOCK_TUNE_TC_SCHEDULE:
+            if (value < 0 || value > 2) return fail(ctx, DOCK_E_INVALID_ARG, "tc schedule must be 0, 1 or 2");
+            ctx->tc_sched = (int)value;
+            return DOCK_OK;
         case DOCK_TUNE_CAND_CAP:
             if (value < 32 || value > (1 << 20)) return fail(ctx, DOCK_E_INVALID_ARG, "cand cap out of range");
             ctx->cand_cap = (int)value;
@@ -1682,6 +1735,9 @@ dock_status dock_get_info(const dock_ctx* ctx, dock_info* info)
         info->sp_row_last = ctx->sp_tx_last;
         info->sp_zt_last = ctx->sp_zt_last;
     }
+    info->tc_ksteps_exec_last = -1.0;
+    if (ctx->tc_variant_last == 1 && ctx->tc_blocks_last > 0 && !info->pending)
+        info->tc_ksteps_exec_last = double((unsigned)ctx->h_small[3]) / ctx->tc_blocks_last;
     return DOCK_OK;
 }
 
@@ -1755,7 +1811,7 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
     unsigned int* cand_max = reinterpret_cast<unsigned int*>(ctx->d_small + 2);
     dk::k_reset<<<(n_units + 255) / 256, 256, 0, ctx->stream>>>(
         static_cast<unsigned long long*>(ctx->T.p), static_cast<unsigned long long*>(ctx->mu.p),
-        static_cast<unsigned int*>(ctx->cnt.p), n_units, fb_cnt, cand_max);
+        static_cast<unsigned int*>(ctx->cnt.p), n_units, fb_cnt, cand_max, reinterpret_cast<unsigned*>(ctx->d_small + 3));
     CU(cudaGetLastError());
     ctx->kernels_last++;
 

@@ -822,7 +822,7 @@ __global__ void k_gather_probes(const ProbeSrc* __restrict__ tab, int n_probes, 
 
 #ifndef DOCK_LAUNCHER_TU   // defined once, in dock.cu
 __global__ void k_reset(unsigned long long* T, unsigned long long* mu, unsigned int* cnt, int n,
-                        unsigned int* fb_cnt, unsigned int* cand_max)
+                        unsigned int* fb_cnt, unsigned int* cand_max, unsigned int* ksum)
 {
     int i = blockIdx.x * blockDim.x + threadIdx.x;
     if (i < n) {
@@ -833,6 +833,7 @@ __global__ void k_reset(unsigned long long* T, unsigned long long* mu, unsigned 
     if (i == 0) {
         *fb_cnt = 0;
         *cand_max = 0;
+        *ksum = 0;
     }
 }
 #endif

@@ -24,6 +24,9 @@
 #pragma once
 #include <cuda_bf16.h>
 
+#include <type_traits>
+#include <utility>
+
 #include "dock_kernels.cuh"
 
 namespace tc {
@@ -60,6 +63,11 @@ struct TcArgs {
                                 // launches: the last CTA to finish resets them)
     int nsteps;                 // K-steps of A per tile (all passes / units, padded to whole ring stages)
     const unsigned char* W;     // [block][step][WCHUNK]
+    // variant 1 occupancy schedule (k_tc_block_tables): per rotation block only the K-steps where some
+    // rotation of the block has a nonzero probe weight (plus zero-weight padding to whole ring stages)
+    const int4* kinfo;          // [block]: (ring stages of the compacted A stream, -, active K-step mask lo, hi)
+    const int* perm;            // [block * ROT]: block position -> unit slot (occupancy clustering); nullptr =
+                                // identity
     int box_bytes;              // bytes of one receptor TMA box (variant 1: the main box; variant 2: one z-plane)
     int box_bytes_pair;         // variant 1: bytes of the pair box
     int rec_stage_bytes;        // variant 1: offset of the pair box; variant 2: one receptor ring slot (unit)
@@ -386,6 +394,18 @@ __host__ __device__ constexpr int pair_txb(int m, int ntt = NT)
 // NT + 4*MXQ - 2 (slot x already holds voxel x + 1) -- at m = 4 the 448 B saved let a 7th weight stage fit.
 __host__ __device__ constexpr int main_box_txb(int m) { return NT + (m + 1) / 2 * 2 - 1; }
 __host__ __device__ constexpr int pair_box_txb(int m) { return NT + 4 * ((m + 3) / 4) - 2; }
+// compile-time loop: f(std::integral_constant<int, i>) for i in [0, N)
+template <class F, int... I>
+__device__ __forceinline__ void static_for_impl(F&& f, std::integer_sequence<int, I...>)
+{
+    (f(std::integral_constant<int, I>{}), ...);
+}
+template <int N, class F>
+__device__ __forceinline__ void static_for(F&& f)
+{
+    static_for_impl(f, std::make_integer_sequence<int, N>{});
+}
+
 // Byte offset of K-step s inside the PAIR pass-1 box ((hi,lo) voxels, 2 per K-step) and pass-2 box
 // ((hi(x),hi(x+1)) slots, 4 voxels per K-step); padding steps (zero weights) re-read the last real
 // step's voxels.
@@ -410,6 +430,9 @@ __host__ __device__ constexpr uint32_t pair_off2(int m, int s, uint32_t row16, u
 // whole boxes (all m z-planes, Q = 4 rows + halo) are resident; the main box is released after pass 1
 // and the pair box after pass 2, so one buffer of each gives full TMA/MMA overlap.  One TMEM buffer of
 // Q x 128 columns; rows are released one by one by the epilogue and restarted in that order.
+// Occupancy schedule: a ring stage (KS K-steps) whose weights are zero for all 128 rotations of the block would
+// add exact zeros to every accumulator; the block's stage mask (k_tc_block_tables) skips it, and the weight
+// stream holds only the block's active stages.  The schedule stays fully unrolled (immediate receptor offsets).
 template <int M, bool GRID>
 __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__ CUtensorMap tmap,
                                                           const __grid_constant__ CUtensorMap tmap_pair, const TcArgs a)
@@ -597,13 +620,15 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                 if (a.chunk > 0) c = fetch();   // one chunk of lookahead: the atomic hides behind the stream
                 n_tiles += n;
                 if (lane == 0) {
-                    const unsigned char* wsrc = a.W + static_cast<size_t>(g / a.ntiles) * NSTEPS * WCHUNK;
+                    const long long blk = g / a.ntiles;
+                    const unsigned char* wsrc = a.W + static_cast<size_t>(blk) * NSTEPS * WCHUNK;
+                    const int nst = a.kinfo[blk].x;   // the block's active stages (compacted weight stream)
                     for (int ti = 0; ti < n; ti++) {
-                        for (int s = 0; s < NSTEPS; s += KS) {
+                        for (int st = 0; st < nst; st++) {
                             if (wuse >= a.wstages) twait(&w_empty[ws], wph ^ 1, tr, tw0);
                             dk::mbar_arrive_expect_tx(&w_full[ws], STAGE);
                             dk::bulk_load(w_smem + static_cast<size_t>(ws) * STAGE,
-                                          wsrc + static_cast<size_t>(s) * WCHUNK, STAGE, &w_full[ws]);
+                                          wsrc + static_cast<size_t>(st) * STAGE, STAGE, &w_full[ws]);
                             wuse++;
                             if (++ws == a.wstages) {
                                 ws = 0;
@@ -691,8 +716,27 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                         }
                 };
                 int ti = 0;   // tiles so far (buffer phases)
-                long long g;
-                for (int n; (n = take_chunk(g, true)) > 0;)
+                long long g, mblk = -1;
+                unsigned long long smk = ~0ull;   // the block's active stages: bit st = dense stage st
+                constexpr int NSTG = NS1 + NS2;
+                constexpr bool MASKED = NSTG <= 64;   // stage masks are one 64-bit word (m <= 6); else dense
+                constexpr unsigned long long HEADM = (1ull << D) - 1ull;
+                // stage st active / active stages before st (dense when unmasked)
+                auto act = [&](int st) -> bool { return !MASKED || ((smk >> (st & 63)) & 1ull); };
+                auto below = [&](unsigned long long mk, int st) -> int {
+                    return MASKED ? __popcll(mk & ((1ull << (st & 63)) - 1ull)) : st;
+                };
+                for (int n; (n = take_chunk(g, true)) > 0;) {
+                    const long long blk = g / a.ntiles;
+                    if (MASKED && blk != mblk) {
+                        const int4 inf = a.kinfo[blk];
+                        smk = static_cast<unsigned long long>(static_cast<uint32_t>(inf.z)) |
+                              (static_cast<unsigned long long>(static_cast<uint32_t>(inf.w)) << 32);
+                        mblk = blk;
+                    }
+                    const int nh = MASKED ? __popcll(smk & HEADM) : D;                 // active head stages
+                    const unsigned long long tmk = MASKED ? smk >> ((NSTG - D) & 63) : ~0ull;   // tail stages
+                    const int nt = MASKED ? __popcll(tmk & HEADM) : D;
                 for (int j = 0; j < n; j++, ti++) {
                     twait(&rec_full[0], ti & 1, tr, tw2);
                     tc_fence_after();
@@ -705,8 +749,10 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                         }
 #pragma unroll
                         for (int st = 0; st < D; st++) {
+                            if (!act(st)) continue;
+                            const int rk = below(smk, st);   // ring stages before it
                             uint32_t ph;
-                            const uint32_t sl = slot_of(st, ph);
+                            const uint32_t sl = slot_of(rk, ph);
                             if (q == 0) {
                                 twait(&w_full[sl], ph, tr, tw1);
                                 tc_fence_after();
@@ -716,30 +762,33 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                             for (int ks = 0; ks < KS; ks++)
                                 umma_bf16(tmem + q * NT, da0 + ((ks * WCHUNK) >> 4),
                                           dB0 + ((pair_off1(M, st * KS + ks, ROW16, ROWTY) + q * ROW16) >> 4), idesc,
-                                          (st == 0 && ks == 0) ? 0u : 1u);
+                                          (rk == 0 && ks == 0) ? 0u : 1u);
                         }
                     }
-#pragma unroll
-                    for (int st = 0; st < D; st++) {
+                    for (int i = 0; i < nh; i++) {
                         uint32_t ph;
-                        umma_commit(&w_empty[slot_of(st, ph)]);
+                        umma_commit(&w_empty[slot_of(i, ph)]);
                     }
-                    advance(D);
+                    advance(nh);
+                    int nact = nh;   // active stages issued so far in this tile (0: the next one overwrites)
                     // pass 1, stages [D, NS1): all rows per stage
 #pragma unroll
                     for (int st = D; st < NS1; st++) {
+                        if (!act(st)) continue;
                         twait(&w_full[ws], wph, tr, tw1);
                         tc_fence_after();
                         const uint64_t da0 = dA0 + ((ws * STAGE) >> 4);
+                        const uint32_t acc0 = nact == 0 ? 0u : 1u;
 #pragma unroll
                         for (int ks = 0; ks < KS; ks++)
 #pragma unroll
                             for (int q = 0; q < Q; q++)
                                 umma_bf16(tmem + q * NT, da0 + ((ks * WCHUNK) >> 4),
                                           dB0 + ((pair_off1(M, st * KS + ks, ROW16, ROWTY) + q * ROW16) >> 4), idesc,
-                                          1u);
+                                          ks == 0 ? acc0 : 1u);
                         umma_commit(&w_empty[ws]);
                         advance(1);
+                        nact++;
                     }
                     umma_commit(&rec_empty[0]);
                     twait(&rec_full[1], ti & 1, tr, tw2);
@@ -747,27 +796,32 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                     // pass 2, stages [0, NS2 - D): all rows per stage
 #pragma unroll
                     for (int st = 0; st < NS2 - D; st++) {
+                        if (!act(NS1 + st)) continue;
                         twait(&w_full[ws], wph, tr, tw1);
                         tc_fence_after();
                         const uint64_t da0 = dA0 + ((ws * STAGE) >> 4);
+                        const uint32_t acc0 = nact == 0 ? 0u : 1u;
 #pragma unroll
                         for (int ks = 0; ks < KS; ks++)
 #pragma unroll
                             for (int q = 0; q < Q; q++)
                                 umma_bf16(tmem + q * NT, da0 + ((ks * WCHUNK) >> 4),
                                           dP0 + ((pair_off2(M, st * KS + ks, ROW16P, ROWTYP) + q * ROW16P) >> 4), idesc,
-                                          1u);
+                                          ks == 0 ? acc0 : 1u);
                         umma_commit(&w_empty[ws]);
                         advance(1);
+                        nact++;
                     }
                     // pass 2, stages [NS2 - D, NS2): row by row; row q is complete after its block
 #pragma unroll
                     for (int q = 0; q < Q; q++) {
 #pragma unroll
                         for (int j = 0; j < D; j++) {
+                            if (MASKED && !((tmk >> j) & 1ull)) continue;
                             const int st = NS2 - D + j;
+                            const int rk = below(tmk, j);
                             uint32_t ph;
-                            const uint32_t sl = slot_of(j, ph);
+                            const uint32_t sl = slot_of(rk, ph);
                             if (q == 0) {
                                 twait(&w_full[sl], ph, tr, tw1);
                                 tc_fence_after();
@@ -777,17 +831,17 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                             for (int ks = 0; ks < KS; ks++)
                                 umma_bf16(tmem + q * NT, da0 + ((ks * WCHUNK) >> 4),
                                           dP0 + ((pair_off2(M, st * KS + ks, ROW16P, ROWTYP) + q * ROW16P) >> 4), idesc,
-                                          1u);
+                                          (nact + rk == 0 && ks == 0) ? 0u : 1u);
                         }
                         umma_commit(&tm_full[q]);
                     }
-#pragma unroll
-                    for (int j = 0; j < D; j++) {
+                    for (int i = 0; i < nt; i++) {
                         uint32_t ph;
-                        umma_commit(&w_empty[slot_of(j, ph)]);
+                        umma_commit(&w_empty[slot_of(i, ph)]);
                     }
-                    advance(D);
+                    advance(nt);
                     umma_commit(&rec_empty[1]);
+                }
                 }
                 if (tr) {
                     atomicAdd(&a.trace[TR_MMA_TOTAL], static_cast<unsigned long long>(clock64() - tstart));
@@ -832,8 +886,9 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                     th = __int_as_float(0x7f800000);
                     th_t = 0xffffffffu;
                     cur = blk;
-                    slot = static_cast<int>(blk) * ROT + r;
-                    rot_ok = slot < n_eff;
+                    const int pos = static_cast<int>(blk) * ROT + r;   // position in the block order
+                    rot_ok = pos < n_eff;
+                    slot = (a.perm && rot_ok) ? a.perm[pos] : pos;     // the unit it holds
                 }
                 const int t0 = static_cast<int>(g % a.ntiles);
                 int tx = t0 % a.ntx, ty = (t0 / a.ntx) % a.nty, tz = t0 / (a.ntx * a.nty);
@@ -1226,29 +1281,222 @@ __global__ void k_pack_receptor_pair_tc(const float* __restrict__ R, uint16_t* _
 }
 #endif
 
-// PAIR scheme A operand: steps [0, S1p) = pass 1 chunks (Whi(vx), Whi(vx)), vx = 2 vxp + c;
-// steps [S1p, S1p + S2p) = pass 2 chunks (Wlo(vx0), Wlo(vx0 + 1)), vx0 = 4 vxq + 2c; padding = 0.
-#ifndef DOCK_LAUNCHER_TU   // defined once, in dock.cu
-__global__ void k_pack_weights_tc_pair(const float* __restrict__ Lw, unsigned char* __restrict__ W, int n_slots, int P,
-                                       int m, int S1, int S1p, int S2, int S2p)
+// ------------------------------------------------------------------ variant 1: occupancy schedule
+//
+// Dense K-steps of variant 1 (k_corr_tc): s in [0, S1) = pass 1 (vz, vy, vxp): voxels vx = 2 vxp, 2 vxp + 1 of
+// the (hi, lo) box; [S1, S1p) padding; s in [S1p, S1p + S2) = pass 2 (vz, vy, vxq): voxels 4 vxq .. 4 vxq + 3
+// of the pair box; the rest padding.  Ring stage st = dense K-steps [st KS, st KS + KS).  A probe grid has at
+// most one occupied voxel per atom, so most stages of one rotation carry only zero weights; a stage
+// whose weights are zero for all 128 rotations of a block adds exact zeros to every accumulator and is skipped by
+// the block.  Units are first grouped into blocks with few distinct active stages (k_tc_cluster).  Stage masks
+// are one 64-bit word (S1p + S2p <= 256, i.e. m <= 6).
+
+// stage bits of an occupied probe voxel (vz, vy, vx)
+__host__ __device__ inline unsigned long long tc1_voxel_stages(int vz, int vy, int vx, int m)
 {
-    const int MXP = (m + 1) / 2, MXQ = (m + 3) / 4, m3 = m * m * m, nsteps = S1p + S2p;
+    const int mxp = (m + 1) / 2, mxq = (m + 3) / 4, s1p = (m * m * mxp + KSTEPS - 1) / KSTEPS * KSTEPS;
+    const int s1 = (vz * m + vy) * mxp + vx / 2, s2 = s1p + (vz * m + vy) * mxq + vx / 4;
+    return (1ull << (s1 / KSTEPS)) | (1ull << (s2 / KSTEPS));
+}
+
+#ifndef DOCK_LAUNCHER_TU   // defined once, in dock.cu
+// Per unit: bit st = ring stage st carries a nonzero folded weight of this unit.
+__global__ void k_tc_unit_masks(const float* __restrict__ Lw, int n_slots, int P, int m,
+                                unsigned long long* __restrict__ masks)
+{
+    const int u = blockIdx.x * blockDim.x + threadIdx.x;
+    if (u >= n_slots) return;
+    const int m3 = m * m * m;
+    const float* base = Lw + static_cast<size_t>(u / dk::RB) * P * m3 * dk::RB + u % dk::RB;
+    unsigned long long sm = 0;
+    for (int v = 0; v < m3; v++) {
+        bool on = false;
+        for (int p = 0; p < P; p++) on = on || base[(static_cast<size_t>(p) * m3 + v) * dk::RB] != 0.f;
+        if (on) sm |= tc1_voxel_stages(v / (m * m), (v / m) % m, v % m, m);
+    }
+    masks[u] = sm;
+}
+
+// Greedy grouping of the units of one window (CL_W units, one CTA) into blocks of ROT: a block takes every
+// remaining unit whose K-steps are already in its union, then the unit that adds the fewest new K-steps (ties:
+// lowest index), until it holds ROT units.  One pass over the window per added unit that grows the union.
+// Measured on the prod workload: the blocks' unions cover 50 % of the K-steps, against 89 % for blocks of
+// consecutive units (the rotations of one probe).  perm[w0 + i] = the unit at block position w0 + i.
+constexpr int CL_THREADS = 1024;
+constexpr int CL_PER = 8;
+constexpr int CL_W = CL_THREADS * CL_PER;   // units per window (a multiple of ROT)
+static_assert(CL_W % ROT == 0, "windows hold whole blocks");
+__global__ void __launch_bounds__(CL_THREADS, 1) k_tc_cluster(const unsigned long long* __restrict__ masks, int n_slots,
+                                                              int* __restrict__ perm)
+{
+    constexpr int NW = CL_THREADS / 32;
+    static_assert(CL_PER == 8 && NW == 32, "the warp-redundant scan assumes 8 x 32 counters");
+    __shared__ unsigned s_cnt[2][CL_PER][NW];   // zero-cost units per (slot k, warp), double-buffered by pass
+    __shared__ unsigned s_min[2][NW];           // per-warp argmin key (added K-steps << 16 | window index)
+    __shared__ unsigned long long s_U[2];       // union of the open block (state double-buffered by pass)
+    __shared__ int s_fill[2], s_out[2], s_left[2];
+    const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
+    const int w0 = blockIdx.x * CL_W;
+    const int n = min(CL_W, n_slots - w0);
+    unsigned long long mk[CL_PER];
+    unsigned live = 0;   // bit k: unit tid + k * CL_THREADS not yet placed
+#pragma unroll
+    for (int k = 0; k < CL_PER; k++) {
+        const int j = tid + k * CL_THREADS;
+        mk[k] = j < n ? masks[w0 + j] : 0ull;
+        if (j < n) live |= 1u << k;
+    }
+    if (tid == 0) {
+        s_U[0] = 0ull;
+        s_fill[0] = 0;
+        s_out[0] = 0;
+        s_left[0] = n;
+    }
+    __syncthreads();
+    for (int ps = 0;; ps ^= 1) {
+        const unsigned long long U = s_U[ps];
+        const int fill = s_fill[ps], out = s_out[ps], left = s_left[ps];
+        if (left <= 0) break;
+        // 1. zero-cost units (a ballot per slot k) and this warp's cheapest positive unit
+        unsigned zb[CL_PER];
+        unsigned best = 0xffffffffu;
+#pragma unroll
+        for (int k = 0; k < CL_PER; k++) {
+            const bool lv = (live >> k) & 1u;
+            const unsigned add = static_cast<unsigned>(__popcll(mk[k] & ~U));
+            zb[k] = __ballot_sync(0xffffffffu, lv && add == 0u);
+            if (lv && add != 0u) best = min(best, (add << 16) | static_cast<unsigned>(tid + k * CL_THREADS));
+            if (lane == 0) s_cnt[ps][k][warp] = __popc(zb[k]);
+        }
+        best = __reduce_min_sync(0xffffffffu, best);
+        if (lane == 0) s_min[ps][warp] = best;
+        __syncthreads();
+        // 2. warp-redundant exclusive scan of the counters in (k, warp) order and argmin over the warps
+        unsigned c8[8], loc = 0;
+#pragma unroll
+        for (int e = 0; e < 8; e++) {
+            c8[e] = s_cnt[ps][lane >> 2][(lane & 3) * 8 + e];
+            loc += c8[e];
+        }
+        unsigned incl = loc;
+#pragma unroll
+        for (int d = 1; d < 32; d <<= 1) {
+            const unsigned t = __shfl_up_sync(0xffffffffu, incl, d);
+            if (lane >= d) incl += t;
+        }
+        const int total = static_cast<int>(__shfl_sync(0xffffffffu, incl, 31));
+        unsigned sel = incl - loc;   // exclusive prefix of counter (lane >> 2, (lane & 3) * 8 + (warp & 7))
+#pragma unroll
+        for (int e = 0; e < 8; e++)
+            if (e < (warp & 7)) sel += c8[e];
+        const unsigned win = __reduce_min_sync(0xffffffffu, s_min[ps][lane]);
+        const int cap = ROT - fill;
+        const int taken = min(total, cap);
+#pragma unroll
+        for (int k = 0; k < CL_PER; k++) {
+            const int base = static_cast<int>(__shfl_sync(0xffffffffu, sel, k * 4 + (warp >> 3)));
+            if ((zb[k] >> lane) & 1u) {
+                const int rank = base + __popc(zb[k] & ((1u << lane) - 1u));
+                if (rank < cap) {
+                    perm[w0 + out + fill + rank] = w0 + tid + k * CL_THREADS;
+                    live &= ~(1u << k);
+                }
+            }
+        }
+        const int nf = fill + taken;
+        const bool add_win = nf < ROT && win != 0xffffffffu;
+        const int jw = static_cast<int>(win & 0xffffu);
+        if (add_win && jw % CL_THREADS == tid) {
+            live &= ~(1u << (jw / CL_THREADS));
+            perm[w0 + out + nf] = w0 + jw;
+        }
+        if (tid == 0) {   // next pass's state (the other buffer: this pass's is still being read)
+            const int nf2 = nf + (add_win ? 1 : 0);
+            s_left[ps ^ 1] = left - taken - (add_win ? 1 : 0);
+            if (nf2 == ROT || s_left[ps ^ 1] == 0) {   // block closed
+                s_out[ps ^ 1] = out + ROT;
+                s_fill[ps ^ 1] = 0;
+                s_U[ps ^ 1] = 0ull;
+            } else {
+                s_out[ps ^ 1] = out;
+                s_fill[ps ^ 1] = nf2;
+                s_U[ps ^ 1] = add_win ? (U | __ldg(&masks[w0 + jw])) : U;
+            }
+        }
+        __syncthreads();
+    }
+}
+
+// Per rotation block (one CTA of 128 threads): the mask of active ring stages -- those with a nonzero weight for
+// some live rotation of the block; at least one, so every row's accumulators are written -- its stage count and
+// the dense stage of every compacted A stage (ksrc).  dense = 1: every stage (occupancy off).  Rotations at
+// positions >= the live count (device-driven fallback) are ignored.  ksum accumulates the executed K-steps.
+__global__ void k_tc_block_tables(const float* __restrict__ Lw, const int* __restrict__ perm, int n_slots,
+                                  const unsigned* __restrict__ n_live, int P, int m, int nsteps, int dense,
+                                  uint16_t* __restrict__ ksrc, int4* __restrict__ kinfo, unsigned* __restrict__ ksum)
+{
+    __shared__ unsigned long long s_mk;
+    const int m3 = m * m * m, blk = blockIdx.x, nstg = nsteps / KSTEPS;
+    uint16_t* src = ksrc + static_cast<size_t>(blk) * nsteps;
+    const int n_eff = n_live ? min(n_slots, static_cast<int>(*n_live)) : n_slots;
+    if (threadIdx.x == 0) s_mk = 0ull;
+    __syncthreads();
+    unsigned long long mk = 0;
+    if (!dense) {
+        for (int r = threadIdx.x; r < ROT; r += blockDim.x) {
+            const int pos = blk * ROT + r;
+            if (pos >= n_eff) continue;
+            const int u = perm ? perm[pos] : pos;
+            const float* base = Lw + static_cast<size_t>(u / dk::RB) * P * m3 * dk::RB + u % dk::RB;
+            for (int v = 0; v < m3; v++) {
+                bool on = false;
+                for (int p = 0; p < P; p++) on = on || base[(static_cast<size_t>(p) * m3 + v) * dk::RB] != 0.f;
+                if (on) mk |= tc1_voxel_stages(v / (m * m), (v / m) % m, v % m, m);
+            }
+        }
+    } else {
+        mk = nstg >= 64 ? ~0ull : (1ull << nstg) - 1ull;
+    }
+    atomicOr(&s_mk, mk);
+    __syncthreads();
+    if (threadIdx.x != 0) return;
+    mk = s_mk;
+    if (mk == 0ull) mk = 1ull;   // all-zero block: one zero-weight stage writes the accumulators
+    int i = 0;
+    for (int st = 0; st < nstg; st++)
+        if ((mk >> st) & 1ull) src[i++] = static_cast<uint16_t>(st);
+    kinfo[blk] = make_int4(i, 0, static_cast<int>(static_cast<uint32_t>(mk)), static_cast<int>(static_cast<uint32_t>(mk >> 32)));
+    if (ksum) atomicAdd(ksum, static_cast<unsigned>(i * KSTEPS));
+}
+
+// Variant 1 A operand, compacted: entry i of block b = dense K-step ksrc[b][i] of the units at the block's
+// positions.  Pass 1 chunks (Whi(vx), Whi(vx)), vx = 2 vxp + c; pass 2 chunks (Wlo(vx0), Wlo(vx0 + 1)),
+// vx0 = 4 vxq + 2c; padding steps are zero.
+__global__ void k_pack_weights_tc1(const float* __restrict__ Lw, const int* __restrict__ perm,
+                                   const uint16_t* __restrict__ ksrc, const int4* __restrict__ kinfo,
+                                   unsigned char* __restrict__ W, int n_slots, int P, int m, int stride)
+{
+    const int MXP = (m + 1) / 2, MXQ = (m + 3) / 4, m3 = m * m * m, S1 = m * m * MXP, S2 = m * m * MXQ;
+    const int S1P = (S1 + KSTEPS - 1) / KSTEPS * KSTEPS;
     const long long n_blocks = (n_slots + ROT - 1) / ROT;
-    const long long total = n_blocks * nsteps * 2 * ROT;
+    const long long total = n_blocks * stride * 2 * ROT;
     for (long long i = blockIdx.x * static_cast<long long>(blockDim.x) + threadIdx.x; i < total;
          i += static_cast<long long>(gridDim.x) * blockDim.x) {
         const int r = static_cast<int>(i % ROT);
         const int c = static_cast<int>((i / ROT) % 2);
-        const int s = static_cast<int>((i / (2 * ROT)) % nsteps);
-        const long long blk = i / (2LL * ROT * nsteps);
-        const long long slot = blk * ROT + r;
+        const int e = static_cast<int>((i / (2 * ROT)) % stride);
+        const long long blk = i / (2LL * ROT * stride);
+        if (e >= kinfo[blk].x * KSTEPS) continue;   // beyond the block's schedule: never streamed
+        const long long pos = blk * ROT + r;
+        const int s = ksrc[blk * stride + e / KSTEPS] * KSTEPS + e % KSTEPS;   // dense K-step
         uint16_t out[8] = {0, 0, 0, 0, 0, 0, 0, 0};
-        auto wval = [&](int vz, int vy, int vx, int p) -> float {
-            if (vx >= m || p >= P) return 0.f;
-            const int v = (vz * m + vy) * m + vx;
-            return Lw[((static_cast<size_t>(slot / dk::RB) * P + p) * m3 + v) * dk::RB + slot % dk::RB];
-        };
-        if (slot < n_slots) {
+        if (pos < n_slots && (s < S1 || (s >= S1P && s < S1P + S2))) {
+            const long long slot = perm ? perm[pos] : pos;
+            auto wval = [&](int vz, int vy, int vx, int p) -> float {
+                if (vx >= m || p >= P) return 0.f;
+                const int v = (vz * m + vy) * m + vx;
+                return Lw[((static_cast<size_t>(slot / dk::RB) * P + p) * m3 + v) * dk::RB + slot % dk::RB];
+            };
             if (s < S1) {
                 const int vxp = s % MXP, vy = (s / MXP) % m, vz = s / (MXP * m);
                 const int vx = 2 * vxp + c;
@@ -1257,8 +1505,8 @@ __global__ void k_pack_weights_tc_pair(const float* __restrict__ Lw, unsigned ch
                     const __nv_bfloat16 hi = __float2bfloat16_rn(wval(vz, vy, vx, p));
                     out[p] = out[4 + p] = __bfloat16_as_ushort(hi);
                 }
-            } else if (s >= S1p && s - S1p < S2) {
-                const int t = s - S1p;
+            } else {
+                const int t = s - S1P;
                 const int vxq = t % MXQ, vy = (t / MXQ) % m, vz = t / (MXQ * m);
                 const int vx0 = 4 * vxq + 2 * c;
 #pragma unroll

@@ -314,6 +314,68 @@ def test_tc_dynamic_scheduler_across_rotation_blocks(D, orc):
     ctx.close()
 
 
+def test_tc_occupancy_schedule_modes(D, orc):
+    """tcgen05 variant 1 runs only the ring stages (4 K-steps) where some rotation of a block has a nonzero
+    weight, after grouping the units into blocks with few distinct active stages (DOCK_TUNE_TC_SCHEDULE 0).
+    Skipped products are exact zeros, so poses (rotation, t_lin and score bits) equal those of the occupancy
+    schedule over consecutive units (1), of the dense schedule (2) and of the exact fallback; the executed
+    K-steps per row do not grow 2 -> 1 -> 0 and the clustered schedule runs fewer than the dense one.  Units of every block validate against the oracle; probes of 0..8 atoms (an empty
+    probe: all-zero blocks run one padding stage)."""
+    P, m = 4, 4
+    R = g.receptor_ftmap_like((48, 40, 37), P)
+    w = g.weights(P)
+    probes = g.probes(6, m, P) + [g.Probe(np.zeros((0, 3)), np.zeros((0, P), np.float32), m)]
+    rot = g.rotations(70)
+    n = len(probes) * len(rot)
+    ctx = _ctx(D, R, w, m, 2)
+
+    def bits(p):
+        return p["rot"], p["t_lin"], p["score"].view(np.uint32)
+
+    out, ks = {}, {}
+    for sched in (2, 1, 0):
+        D.dock_set_tuning(ctx, D.DOCK_TUNE_TC_SCHEDULE, sched)
+        out[sched] = D.dock_probe_batch(ctx, probes, rot, k=4, rho=1)
+        info = D.dock_get_info(ctx)
+        assert info["engine_last"] == 2 and info["tc_variant_last"] == 1
+        ks[sched] = info["tc_ksteps_exec_last"]
+    assert ks[2] == 48.0 and ks[0] <= ks[1] <= ks[2] and ks[0] < ks[2], ks
+    for sched in (1, 0):
+        assert all(np.array_equal(a, b) for a, b in zip(bits(out[sched]), bits(out[2]))), sched
+    D.dock_set_tuning(ctx, D.DOCK_TUNE_FORCE_FALLBACK, 1)
+    fb = D.dock_probe_batch(ctx, probes, rot, k=4, rho=1)
+    D.dock_set_tuning(ctx, D.DOCK_TUNE_FORCE_FALLBACK, 0)
+    assert all(np.array_equal(a, b) for a, b in zip(bits(fb), bits(out[0])))
+    ctx.close()
+    units = sorted({0, 69, 70, 139, 200, 333, 350, 419, n - 70, n - 1})
+    SA = _oracle_units(orc, R, w, probes, rot, units)
+    mism = 0
+    for u, (S, A) in zip(units, SA):
+        assert (out[0][u]["rot"] == u % len(rot)).all()
+        mism += validate_unit(S, A, out[0][u]["t_lin"], out[0][u]["score"], 4, 1)
+    assert mism == 0
+
+
+def test_tc_occupancy_schedule_integer_exact(D, orc):
+    """Clustered occupancy schedule (> 128 units, m = 3 and m = 2) on integer inputs: poses equal the FP64
+    oracle exactly, ties included (P9)."""
+    P = 4
+    R = g.receptor_integer((40, 24, 20), P, lo=-2, hi=2)
+    w = g.weights_integer(P)
+    for m, n_rot in ((3, 60), (2, 50)):
+        probes = g.probes(3, m, P, integer=True)
+        rot = g.rotations(n_rot)
+        ctx = _ctx(D, R, w, m, 2)
+        poses = D.dock_probe_batch(ctx, probes, rot, k=4, rho=1)
+        info = D.dock_get_info(ctx)
+        assert info["tc_variant_last"] == 1 and info["tc_ksteps_exec_last"] > 0
+        ctx.close()
+        t_o, s_o, st = orc.dock(R, w, H, probes, rot, 4, 1)
+        assert (st == 0).all()
+        assert np.array_equal(poses["t_lin"], t_o.astype(np.int32))
+        assert np.array_equal(poses["score"].astype(np.float64), s_o)
+
+
 @pytest.mark.parametrize("engine", ENGINES)
 @pytest.mark.parametrize("rho,k", [(0, 4), (1, 4), (0, 1)])
 def test_integer_inputs_exact_poses(D, orc, rho, k, engine):
