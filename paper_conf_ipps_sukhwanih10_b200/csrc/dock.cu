@@ -101,7 +101,10 @@ struct dock_ctx {
     DevBuf Wtc;
     // variant 1 occupancy schedule of the main pass / of the fallback: K-step tables, source steps, per-block
     // (stages, first pair entry), clustering permutation and unit masks
-    DevBuf tc_ksrc, tc_kinfo, tc_perm, tc_umask, fb_ksrc, fb_kinfo;
+    DevBuf tc_ksrc, tc_kinfo, tc_perm, tc_umask, tc_sorted, fb_ksrc, fb_kinfo, fb_umask, tc_seg, tc_pref;
+    int tc_seg_cost = 8;       // per-tile cost of a chunk beyond its ring stages, in ring stages (prod: 0 / 3 / 6 /
+                               // 9 / 12 / 24 -> 12.20 / 11.79 / 11.40 / 11.35 / 11.48 / 11.84 ms); DOCK_TC_SEG_COST
+                               // (environment) overrides it
     // diagnostics (environment, read at init): DOCK_TC_TRACE=1 prints per-role cycle counters of every
     // tcgen05 launch to stderr
     unsigned long long* d_trace = nullptr;
@@ -1000,22 +1003,38 @@ dock_status pack_weights_tc(dock_ctx* ctx, int m, int v, int n_slots, const floa
         TRY(ensure(ctx, ks, sizeof(uint16_t) * n_blocks * tp.nsteps));
         TRY(ensure(ctx, ki, sizeof(int4) * n_blocks));
         const int* perm = nullptr;
-        if (!fb && ctx->tc_sched == 0 && tp.nsteps <= 64 * tc::KSTEPS && n_slots > tc::ROT) {
-            TRY(ensure(ctx, ctx->tc_umask, sizeof(unsigned long long) * n_slots));
+        const int nstg = tp.nsteps / tc::KSTEPS;
+        const bool masked = ctx->tc_sched != 2 && nstg <= 64;
+        const unsigned long long* um = nullptr;
+        if (masked) {   // per-unit stage masks (positions past the live count: none)
+            TRY(ensure(ctx, fb ? ctx->fb_umask : ctx->tc_umask, sizeof(unsigned long long) * n_slots));
+            auto* umw = static_cast<unsigned long long*>((fb ? ctx->fb_umask : ctx->tc_umask).p);
+            const int warps = (n_slots + dk::RB - 1) / dk::RB;
+            tc::k_tc_unit_masks<<<(warps + 3) / 4, 128, 0, ctx->stream>>>(Lw, n_slots, n_live, ctx->P, m, umw);
+            CU(cudaGetLastError());
+            ctx->kernels_last++;
+            um = umw;
+        }
+        if (masked && !fb && ctx->tc_sched == 0 && n_slots > tc::ROT) {
             TRY(ensure(ctx, ctx->tc_perm, sizeof(int) * n_blocks * tc::ROT));
-            auto* um = static_cast<unsigned long long*>(ctx->tc_umask.p);
-            tc::k_tc_unit_masks<<<(n_slots + 127) / 128, 128, 0, ctx->stream>>>(Lw, n_slots, ctx->P, m, um);
+            const int windows = (n_slots + tc::CL_W - 1) / tc::CL_W;
+            if (nstg <= tc::CB_BITS) {   // distinct masks fit a histogram
+                TRY(ensure(ctx, ctx->tc_sorted, sizeof(int) * n_slots));
+                const int sm = (int)sizeof(tc::ClusterBinsSmem);
+                CU(cudaFuncSetAttribute(tc::k_tc_cluster_bins, cudaFuncAttributeMaxDynamicSharedMemorySize, sm));
+                tc::k_tc_cluster_bins<<<windows, tc::CL_THREADS, sm, ctx->stream>>>(
+                    um, n_slots, static_cast<int*>(ctx->tc_sorted.p), static_cast<int*>(ctx->tc_perm.p));
+            } else {
+                tc::k_tc_cluster<<<windows, tc::CL_THREADS, 0, ctx->stream>>>(um, n_slots,
+                                                                               static_cast<int*>(ctx->tc_perm.p));
+            }
             CU(cudaGetLastError());
-            tc::k_tc_cluster<<<(n_slots + tc::CL_W - 1) / tc::CL_W, tc::CL_THREADS, 0, ctx->stream>>>(
-                um, n_slots, static_cast<int*>(ctx->tc_perm.p));
-            CU(cudaGetLastError());
-            ctx->kernels_last += 2;
+            ctx->kernels_last++;
             perm = static_cast<const int*>(ctx->tc_perm.p);
         }
-        ctx->tc_perm_on = perm != nullptr;
+        if (!fb) ctx->tc_perm_on = perm != nullptr;
         tc::k_tc_block_tables<<<(int)n_blocks, 128, 0, ctx->stream>>>(
-            Lw, perm, n_slots, n_live, ctx->P, m, tp.nsteps, (ctx->tc_sched == 2 || tp.nsteps > 64 * tc::KSTEPS) ? 1 : 0,
-            static_cast<uint16_t*>(ks.p), static_cast<int4*>(ki.p),
+            um, perm, n_slots, tp.nsteps, static_cast<uint16_t*>(ks.p), static_cast<int4*>(ki.p),
             fb ? nullptr : reinterpret_cast<unsigned*>(ctx->d_small + 3));
         CU(cudaGetLastError());
         tc::k_pack_weights_tc1<<<grid, 256, 0, ctx->stream>>>(Lw, perm, static_cast<const uint16_t*>(ks.p),
@@ -1120,7 +1139,7 @@ dock_status run_grid_tc(dock_ctx* ctx, int m, int n_slots, const float* Lw, floa
 struct FbKey {   // everything the captured fallback graph bakes in (compared bytewise)
     int m, kind, v, G, k, rho, ch, nepi, P, nx, ny, nz;
     int sp_nat, sp_npl, sp_smem, sp_xts;
-    const void *fb_list, *d_small, *dyn, *grid, *Lw, *W, *picks, *slots, *ctl, *w, *ksrc, *kinfo;
+    const void *fb_list, *d_small, *dyn, *grid, *Lw, *W, *picks, *slots, *ctl, *w, *ksrc, *kinfo, *umask;
     const void *spG, *sp_tv, *sp_ts, *sp_nt, *sp_dw, *sp_sa, *fb_groups;
 };
 static_assert(sizeof(FbKey) <= sizeof(((dock_ctx*)nullptr)->fb_key), "fb_key too small");
@@ -1313,6 +1332,7 @@ dock_status launch_fallback(dock_ctx* ctx, int m, int kind, int k, int rho, cons
         const TcPlan& tp = ctx->tcplan[vv][m];
         TRY(ensure(ctx, ctx->fb_W, (size_t)tp.nsteps * tc::WCHUNK));
         TRY(ensure(ctx, ctx->fb_ksrc, sizeof(uint16_t) * tp.nsteps));
+        TRY(ensure(ctx, ctx->fb_umask, sizeof(unsigned long long) * ch));
         TRY(ensure(ctx, ctx->fb_kinfo, sizeof(int4)));
     } else if (kind == ENG_FFMA) {
         key.G = choose_regions(ctx, (ch + dk::RB - 1) / dk::RB);
@@ -1333,6 +1353,7 @@ dock_status launch_fallback(dock_ctx* ctx, int m, int kind, int k, int rho, cons
     key.W = ctx->fb_W.p;
     key.ksrc = ctx->fb_ksrc.p;
     key.kinfo = ctx->fb_kinfo.p;
+    key.umask = ctx->fb_umask.p;
     key.picks = ctx->fb_picks.p;
     key.slots = ctx->fb_slots.p;
     key.ctl = ctx->fb_ctl.p;
@@ -1443,7 +1464,8 @@ void dock_destroy(dock_ctx* ctx)
                       &ctx->mu,      &ctx->cnt,      &ctx->cand,   &ctx->poses,    &ctx->fb_list,  &ctx->grid,
                       &ctx->slots,   &ctx->units,    &ctx->Lw_fb,  &ctx->picks,    &ctx->fb_grid,  &ctx->fb_Lw,
                       &ctx->fb_W,    &ctx->fb_picks, &ctx->fb_slots, &ctx->fb_ctl,   &ctx->tc_ksrc,
-                      &ctx->tc_kinfo, &ctx->tc_perm, &ctx->tc_umask, &ctx->fb_ksrc, &ctx->fb_kinfo};
+                      &ctx->tc_kinfo, &ctx->tc_perm, &ctx->tc_umask, &ctx->tc_sorted, &ctx->fb_ksrc, &ctx->fb_kinfo,
+                      &ctx->fb_umask, &ctx->tc_seg,  &ctx->tc_pref};
     for (DevBuf* b : bufs)
         if (b->p) cudaFree(b->p);
     if (ctx->d_trace) cudaFree(ctx->d_trace);
@@ -1516,6 +1538,7 @@ dock_status dock_init(const dock_grid_desc* g, const float* receptor, const floa
     for (auto& st : ctx->stage)
         if (cudaEventCreateWithFlags(&st.ev, cudaEventDisableTiming) != cudaSuccess) return bail(DOCK_E_CUDA);
     if (const char* e = getenv("DOCK_FB_HOST_LOOP")) ctx->fb_host_loop = atoi(e);
+    if (const char* e = getenv("DOCK_TC_SEG_COST")) ctx->tc_seg_cost = std::max(0, atoi(e));   // tuning experiments
     if (const char* e = getenv("DOCK_TC_TRACE")) {
         if (atoi(e) > 0 && cudaMalloc(&ctx->d_trace, sizeof(unsigned long long) * tc::TR_N) != cudaSuccess)
             return bail(DOCK_E_OOM);
@@ -1878,6 +1901,18 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
         ta.cand = candp;
         const int64_t items = tc_ctas(ta, n_units, ctx->n_sms);
         if (items > 0x7fffffff) return fail(ctx, DOCK_E_UNSUPPORTED, "too many work items");
+        if (v == 1 && ta.chunk > 0 && ctx->tc_sched != 2 && n_blocks <= (1 << 16)) {
+            // scheduler segments of equal estimated cost (blocks' occupancy schedules differ in length)
+            TRY(ensure(ctx, ctx->tc_seg, sizeof(long long) * (items + 1)));
+            TRY(ensure(ctx, ctx->tc_pref, sizeof(long long) * n_blocks));
+            const int cpb = (ta.ntiles + ta.chunk - 1) / ta.chunk;
+            tc::k_tc_segments<<<1, 256, 0, ctx->stream>>>(ta.kinfo, (int)n_blocks, cpb, (int)items, ctx->tc_seg_cost,
+                                                          static_cast<long long*>(ctx->tc_pref.p),
+                                                          static_cast<long long*>(ctx->tc_seg.p));
+            CU(cudaGetLastError());
+            ctx->kernels_last++;
+            ta.seg = static_cast<const long long*>(ctx->tc_seg.p);
+        }
         if (ctx->d_trace) CU(cudaMemsetAsync(ctx->d_trace, 0, sizeof(unsigned long long) * tc::TR_N, ctx->stream));
         CU(cudaEventRecord(ctx->ev_corr[0], ctx->stream));
         CU(launch_tc(m, v, false, ctx->tcplan[v][m], ta, (int)items, ctx->stream));

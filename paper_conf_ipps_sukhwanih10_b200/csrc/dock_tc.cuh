@@ -68,6 +68,8 @@ struct TcArgs {
     const int4* kinfo;          // [block]: (ring stages of the compacted A stream, -, active K-step mask lo, hi)
     const int* perm;            // [block * ROT]: block position -> unit slot (occupancy clustering); nullptr =
                                 // identity
+    const long long* seg;       // [gridDim.x + 1]: dynamic scheduler segment boundaries (chunk ids) balanced by the
+                                // blocks' schedule lengths (k_tc_segments); nullptr = equal chunk counts
     int box_bytes;              // bytes of one receptor TMA box (variant 1: the main box; variant 2: one z-plane)
     int box_bytes_pair;         // variant 1: bytes of the pair box
     int rec_stage_bytes;        // variant 1: offset of the pair box; variant 2: one receptor ring slot (unit)
@@ -556,8 +558,13 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
             // (warp-wide: lane 0 streams, all lanes search for chunks to help with)
             // segment j: chunk ids [lo, hi)
             auto seg_range = [&](int j, long long& lo, long long& hi) {
-                lo = static_cast<long long>(j) * n_chunks / NS;
-                hi = static_cast<long long>(j + 1) * n_chunks / NS;
+                if (a.seg) {
+                    lo = a.seg[j];
+                    hi = a.seg[j + 1];
+                } else {
+                    lo = static_cast<long long>(j) * n_chunks / NS;
+                    hi = static_cast<long long>(j + 1) * n_chunks / NS;
+                }
             };
             int seg = blockIdx.x;
             auto fetch = [&]() -> long long {   // next chunk id, -1 when every segment is exhausted
@@ -1299,22 +1306,293 @@ __host__ __device__ inline unsigned long long tc1_voxel_stages(int vz, int vy, i
     return (1ull << (s1 / KSTEPS)) | (1ull << (s2 / KSTEPS));
 }
 
+constexpr int CL_THREADS = 1024;
+constexpr int CL_PER = 8;
+constexpr int CL_W = CL_THREADS * CL_PER;   // units per clustering window (a multiple of ROT)
+static_assert(CL_W % ROT == 0, "windows hold whole blocks");
+
 #ifndef DOCK_LAUNCHER_TU   // defined once, in dock.cu
-// Per unit: bit st = ring stage st carries a nonzero folded weight of this unit.
-__global__ void k_tc_unit_masks(const float* __restrict__ Lw, int n_slots, int P, int m,
-                                unsigned long long* __restrict__ masks)
+// Per unit: bit st = ring stage st carries a nonzero folded weight of this unit.  One warp per register batch
+// of RB = 8 units: lane v reads the 8 units' weights of voxel v (32 contiguous bytes per channel), the stage bits
+// of the occupied voxels are OR-reduced over the warp.  n_live (optional): units at or past it are masked out.
+__global__ void k_tc_unit_masks(const float* __restrict__ Lw, int n_slots, const unsigned* __restrict__ n_live,
+                                int P, int m, unsigned long long* __restrict__ masks)
 {
-    const int u = blockIdx.x * blockDim.x + threadIdx.x;
-    if (u >= n_slots) return;
+    static_assert(dk::RB == 8, "one warp covers the 8 units of a register batch");
+    const int warp = (blockIdx.x * blockDim.x + threadIdx.x) >> 5, lane = threadIdx.x & 31;
+    const int n_eff = n_live ? min(n_slots, static_cast<int>(*n_live)) : n_slots;
+    const int u0 = warp * dk::RB;
+    if (u0 >= n_slots) return;
     const int m3 = m * m * m;
-    const float* base = Lw + static_cast<size_t>(u / dk::RB) * P * m3 * dk::RB + u % dk::RB;
-    unsigned long long sm = 0;
-    for (int v = 0; v < m3; v++) {
-        bool on = false;
-        for (int p = 0; p < P; p++) on = on || base[(static_cast<size_t>(p) * m3 + v) * dk::RB] != 0.f;
-        if (on) sm |= tc1_voxel_stages(v / (m * m), (v / m) % m, v % m, m);
+    const float* base = Lw + static_cast<size_t>(warp) * P * m3 * dk::RB;
+    unsigned long long sm[dk::RB];
+#pragma unroll
+    for (int r = 0; r < dk::RB; r++) sm[r] = 0ull;
+    for (int v = lane; v < m3; v += 32) {
+        unsigned on = 0;   // bit r: unit u0 + r has a nonzero weight at voxel v
+        for (int p = 0; p < P; p++) {
+            const float4* q = reinterpret_cast<const float4*>(base + (static_cast<size_t>(p) * m3 + v) * dk::RB);
+            const float4 w0 = q[0], w1 = q[1];
+            on |= (w0.x != 0.f ? 1u : 0u) | (w0.y != 0.f ? 2u : 0u) | (w0.z != 0.f ? 4u : 0u) | (w0.w != 0.f ? 8u : 0u) |
+                  (w1.x != 0.f ? 16u : 0u) | (w1.y != 0.f ? 32u : 0u) | (w1.z != 0.f ? 64u : 0u) |
+                  (w1.w != 0.f ? 128u : 0u);
+        }
+        if (on) {
+            const unsigned long long st = tc1_voxel_stages(v / (m * m), (v / m) % m, v % m, m);
+#pragma unroll
+            for (int r = 0; r < dk::RB; r++)
+                if ((on >> r) & 1u) sm[r] |= st;
+        }
     }
-    masks[u] = sm;
+#pragma unroll
+    for (int r = 0; r < dk::RB; r++) {
+        const unsigned lo = __reduce_or_sync(0xffffffffu, static_cast<unsigned>(sm[r]));
+        const unsigned hi = __reduce_or_sync(0xffffffffu, static_cast<unsigned>(sm[r] >> 32));
+        if (lane == r && u0 + r < n_slots)
+            masks[u0 + r] = u0 + r < n_eff ? (static_cast<unsigned long long>(hi) << 32) | lo : 0ull;
+    }
+}
+
+// Greedy grouping over distinct masks (stage masks of <= CB_BITS bits, one CTA per window of CL_W units): the
+// window's units are binned by mask (a counting sort); one warp then runs the greedy of
+// k_tc_cluster on the distinct masks -- a block takes every remaining mask already inside its union (all its
+// units, as far as the block has room), then all units of the mask that adds the fewest stages (ties: lowest
+// mask) -- and the take records are expanded into the permutation.  Same blocks as the unit greedy up to the
+// order of equal masks; the passes scale with the distinct masks, not the units.
+constexpr int CB_BITS = 12;
+constexpr int CB_N = 1 << CB_BITS;
+constexpr int CB_MAXREC = CB_N + 2 * (CL_W / ROT);   // distinct masks + two capacity splits per block
+struct ClusterBinsSmem {
+    int hist[CB_N];           // units per mask -> (after the scan) first sorted position of the mask
+    int fill[CB_N];           // stable-rank cursor per mask
+    uint16_t lmask[CB_N];     // distinct masks present
+    int lrem[CB_N];           // their remaining units
+    int lbase[CB_N];          // their first sorted position
+    int rec_src[CB_MAXREC];   // take records: sorted position of the first unit taken
+    int rec_cnt[CB_MAXREC];   //               units taken
+    int rec_pos[CB_MAXREC];   //               block position of the first one
+    uint16_t umask[CL_W];     // the window's unit masks
+};
+__global__ void __launch_bounds__(1024, 1) k_tc_cluster_bins(const unsigned long long* __restrict__ masks, int n_slots,
+                                                             int* __restrict__ sorted, int* __restrict__ perm)
+{
+    extern __shared__ __align__(16) unsigned char cb_raw[];
+    ClusterBinsSmem& S = *reinterpret_cast<ClusterBinsSmem*>(cb_raw);
+    __shared__ int s_nl, s_nrec;
+    const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
+    const int w0 = blockIdx.x * CL_W;
+    const int n = min(CL_W, n_slots - w0);
+    int* srt = sorted + w0;
+    for (int i = tid; i < CB_N; i += blockDim.x) S.hist[i] = 0;
+    __syncthreads();
+    for (int i = tid; i < n; i += blockDim.x) {
+        const int b = static_cast<int>(masks[w0 + i]);
+        S.umask[i] = static_cast<uint16_t>(b);
+        atomicAdd(&S.hist[b], 1);
+    }
+    __syncthreads();
+    if (warp == 0) {
+        // exclusive scan of the histogram (128 bins per lane) and the list of distinct masks, in mask order
+        constexpr int PER = CB_N / 32;
+        int loc = 0, nz = 0;
+        for (int k = 0; k < PER; k++) {
+            loc += S.hist[lane * PER + k];
+            nz += S.hist[lane * PER + k] != 0;
+        }
+        int incl = loc, inz = nz;
+        for (int d = 1; d < 32; d <<= 1) {
+            const int t = __shfl_up_sync(0xffffffffu, incl, d), tz = __shfl_up_sync(0xffffffffu, inz, d);
+            if (lane >= d) {
+                incl += t;
+                inz += tz;
+            }
+        }
+        int run = incl - loc, li = inz - nz;
+        for (int k = 0; k < PER; k++) {
+            const int b = lane * PER + k, c = S.hist[b];
+            S.fill[b] = run;
+            if (c) {
+                S.lmask[li] = static_cast<uint16_t>(b);
+                S.lrem[li] = c;
+                S.lbase[li] = run;
+                li++;
+            }
+            S.hist[b] = run;
+            run += c;
+        }
+        if (lane == 31) s_nl = inz;
+    }
+    __syncthreads();
+    // counting sort by mask (the order among units of equal masks is arbitrary: blocks, stage masks and every
+    // per-rotation result are the same for any order)
+    for (int i = tid; i < n; i += blockDim.x) srt[atomicAdd(&S.fill[S.umask[i]], 1)] = w0 + i;
+    __syncthreads();
+    if (warp == 0 && s_nl <= 32 * 8) {
+        // the greedy over <= 256 distinct masks with the list in registers: lane L owns entries [8L, 8L + 8)
+        constexpr int E = 8;
+        const int nl = s_nl;
+        unsigned msk[E];
+        int rem[E], base[E];
+#pragma unroll
+        for (int e = 0; e < E; e++) {
+            const int j = lane * E + e;
+            msk[e] = j < nl ? static_cast<unsigned>(S.lmask[j]) : 0u;
+            rem[e] = j < nl ? S.lrem[j] : 0;
+            base[e] = j < nl ? S.lbase[j] : 0;
+        }
+        unsigned U = 0;
+        int fill = 0, out = 0, nrec = 0, left = n;
+        while (left > 0) {
+            // zero-cost masks in list order, as many units as fit
+            const int cap = ROT - fill;
+            int cz = 0;
+#pragma unroll
+            for (int e = 0; e < E; e++) cz += (rem[e] > 0 && (msk[e] & ~U) == 0u) ? rem[e] : 0;
+            int incl = cz;
+            for (int d = 1; d < 32; d <<= 1) {
+                const int t = __shfl_up_sync(0xffffffffu, incl, d);
+                if (lane >= d) incl += t;
+            }
+            int before = incl - cz, ntake = 0;
+            int tk[E];
+#pragma unroll
+            for (int e = 0; e < E; e++) {
+                const int c = (rem[e] > 0 && (msk[e] & ~U) == 0u) ? rem[e] : 0;
+                tk[e] = max(0, min(c, cap - before));
+                before += c;
+                ntake += tk[e] > 0;
+            }
+            int rinc = ntake;
+            for (int d = 1; d < 32; d <<= 1) {
+                const int t = __shfl_up_sync(0xffffffffu, rinc, d);
+                if (lane >= d) rinc += t;
+            }
+            int r = nrec + rinc - ntake, pos = out + fill + (incl - cz);
+#pragma unroll
+            for (int e = 0; e < E; e++) {
+                if (tk[e] > 0) {
+                    S.rec_src[r] = base[e];
+                    S.rec_cnt[r] = tk[e];
+                    S.rec_pos[r] = pos;
+                    r++;
+                    rem[e] -= tk[e];
+                    base[e] += tk[e];
+                }
+                pos += tk[e];
+            }
+            nrec += __shfl_sync(0xffffffffu, rinc, 31);
+            const int taken = min(__shfl_sync(0xffffffffu, incl, 31), cap);
+            fill += taken;
+            left -= taken;
+            if (fill < ROT && left > 0) {
+                // the mask that adds the fewest stages (ties: the lowest entry = the lowest mask)
+                unsigned best = 0xffffffffu;
+#pragma unroll
+                for (int e = 0; e < E; e++)
+                    if (rem[e] > 0)
+                        best = min(best, (static_cast<unsigned>(__popc(msk[e] & ~U)) << 16) |
+                                             static_cast<unsigned>(lane * E + e));
+                best = __reduce_min_sync(0xffffffffu, best);
+                const int j = static_cast<int>(best & 0xffffu), owner = j / E, ej = j % E;
+                int take = 0;
+                unsigned mj = 0;
+#pragma unroll
+                for (int e = 0; e < E; e++)
+                    if (lane == owner && e == ej) {
+                        take = min(rem[e], ROT - fill);
+                        S.rec_src[nrec] = base[e];
+                        S.rec_cnt[nrec] = take;
+                        S.rec_pos[nrec] = out + fill;
+                        rem[e] -= take;
+                        base[e] += take;
+                        mj = msk[e];
+                    }
+                take = __shfl_sync(0xffffffffu, take, owner);
+                mj = __shfl_sync(0xffffffffu, mj, owner);
+                nrec++;
+                U |= mj;
+                fill += take;
+                left -= take;
+            }
+            if (fill == ROT || left == 0) {
+                out += ROT;
+                fill = 0;
+                U = 0;
+            }
+        }
+        if (lane == 0) s_nrec = nrec;
+    } else if (warp == 0) {
+        // the greedy over the distinct masks (one warp; list entries lane, lane + 32, ...)
+        const int nl = s_nl;
+        unsigned U = 0;
+        int fill = 0, out = 0, nrec = 0, left = n;
+        while (left > 0) {
+            const int cap = ROT - fill;
+            // zero-cost masks in list order, as many units as fit
+            int taken_before = 0;
+            for (int j0 = 0; j0 < nl && taken_before < cap; j0 += 32) {
+                const int j = j0 + lane;
+                const int rem = j < nl ? S.lrem[j] : 0;
+                const bool z = rem > 0 && (static_cast<unsigned>(S.lmask[j]) & ~U) == 0u;
+                int c = z ? rem : 0, incl = c;
+                for (int d = 1; d < 32; d <<= 1) {
+                    const int t = __shfl_up_sync(0xffffffffu, incl, d);
+                    if (lane >= d) incl += t;
+                }
+                const int before = taken_before + incl - c;
+                const int take = z ? max(0, min(c, cap - before)) : 0;
+                const unsigned tb = __ballot_sync(0xffffffffu, take > 0);
+                if (take > 0) {
+                    const int r = nrec + __popc(tb & ((1u << lane) - 1u));
+                    S.rec_src[r] = S.lbase[j];
+                    S.rec_cnt[r] = take;
+                    S.rec_pos[r] = out + fill + before;
+                    S.lrem[j] = rem - take;
+                    S.lbase[j] += take;
+                }
+                nrec += __popc(tb);
+                taken_before += __shfl_sync(0xffffffffu, incl, 31);
+                taken_before = min(taken_before, cap);
+            }
+            fill += taken_before;
+            left -= taken_before;
+            __syncwarp();
+            if (fill < ROT && left > 0) {
+                // the mask that adds the fewest stages (ties: the lowest mask)
+                unsigned best = 0xffffffffu;
+                for (int j = lane; j < nl; j += 32)
+                    if (S.lrem[j] > 0)
+                        best = min(best, (static_cast<unsigned>(__popc(static_cast<unsigned>(S.lmask[j]) & ~U)) << 16) |
+                                             static_cast<unsigned>(j));
+                best = __reduce_min_sync(0xffffffffu, best);
+                const int j = static_cast<int>(best & 0xffffu);
+                const int take = min(S.lrem[j], ROT - fill);
+                if (lane == 0) {
+                    S.rec_src[nrec] = S.lbase[j];
+                    S.rec_cnt[nrec] = take;
+                    S.rec_pos[nrec] = out + fill;
+                    S.lrem[j] -= take;
+                    S.lbase[j] += take;
+                }
+                __syncwarp();
+                nrec++;
+                U |= static_cast<unsigned>(S.lmask[j]);
+                fill += take;
+                left -= take;
+            }
+            if (fill == ROT || left == 0) {
+                out += ROT;
+                fill = 0;
+                U = 0;
+            }
+        }
+        if (lane == 0) s_nrec = nrec;
+    }
+    __syncthreads();
+    // expand the records: record r places sorted units [src, src + cnt) at block positions [pos, pos + cnt)
+    const int nrec = s_nrec;
+    for (int r = warp; r < nrec; r += blockDim.x / 32)
+        for (int i = lane; i < S.rec_cnt[r]; i += 32) perm[w0 + S.rec_pos[r] + i] = srt[S.rec_src[r] + i];
 }
 
 // Greedy grouping of the units of one window (CL_W units, one CTA) into blocks of ROT: a block takes every
@@ -1322,10 +1600,6 @@ __global__ void k_tc_unit_masks(const float* __restrict__ Lw, int n_slots, int P
 // lowest index), until it holds ROT units.  One pass over the window per added unit that grows the union.
 // Measured on the prod workload: the blocks' unions cover 50 % of the K-steps, against 89 % for blocks of
 // consecutive units (the rotations of one probe).  perm[w0 + i] = the unit at block position w0 + i.
-constexpr int CL_THREADS = 1024;
-constexpr int CL_PER = 8;
-constexpr int CL_W = CL_THREADS * CL_PER;   // units per window (a multiple of ROT)
-static_assert(CL_W % ROT == 0, "windows hold whole blocks");
 __global__ void __launch_bounds__(CL_THREADS, 1) k_tc_cluster(const unsigned long long* __restrict__ masks, int n_slots,
                                                               int* __restrict__ perm)
 {
@@ -1427,46 +1701,89 @@ __global__ void __launch_bounds__(CL_THREADS, 1) k_tc_cluster(const unsigned lon
     }
 }
 
-// Per rotation block (one CTA of 128 threads): the mask of active ring stages -- those with a nonzero weight for
-// some live rotation of the block; at least one, so every row's accumulators are written -- its stage count and
-// the dense stage of every compacted A stage (ksrc).  dense = 1: every stage (occupancy off).  Rotations at
-// positions >= the live count (device-driven fallback) are ignored.  ksum accumulates the executed K-steps.
-__global__ void k_tc_block_tables(const float* __restrict__ Lw, const int* __restrict__ perm, int n_slots,
-                                  const unsigned* __restrict__ n_live, int P, int m, int nsteps, int dense,
-                                  uint16_t* __restrict__ ksrc, int4* __restrict__ kinfo, unsigned* __restrict__ ksum)
+// Per rotation block (one CTA of 128 threads): the mask of active ring stages -- the OR of its units' masks
+// (k_tc_unit_masks: zero for positions past the live count); at least one stage, so every row's accumulators are
+// written -- its stage count and the dense stage of every compacted A stage (ksrc).  masks == nullptr: every
+// stage (dense schedule).  ksum accumulates the executed K-steps (statistics).
+__global__ void k_tc_block_tables(const unsigned long long* __restrict__ masks, const int* __restrict__ perm,
+                                  int n_slots, int nsteps, uint16_t* __restrict__ ksrc, int4* __restrict__ kinfo,
+                                  unsigned* __restrict__ ksum)
 {
-    __shared__ unsigned long long s_mk;
-    const int m3 = m * m * m, blk = blockIdx.x, nstg = nsteps / KSTEPS;
+    const int blk = blockIdx.x, nstg = nsteps / KSTEPS, lane = threadIdx.x & 31;
     uint16_t* src = ksrc + static_cast<size_t>(blk) * nsteps;
-    const int n_eff = n_live ? min(n_slots, static_cast<int>(*n_live)) : n_slots;
-    if (threadIdx.x == 0) s_mk = 0ull;
-    __syncthreads();
     unsigned long long mk = 0;
-    if (!dense) {
+    if (masks) {
         for (int r = threadIdx.x; r < ROT; r += blockDim.x) {
             const int pos = blk * ROT + r;
-            if (pos >= n_eff) continue;
-            const int u = perm ? perm[pos] : pos;
-            const float* base = Lw + static_cast<size_t>(u / dk::RB) * P * m3 * dk::RB + u % dk::RB;
-            for (int v = 0; v < m3; v++) {
-                bool on = false;
-                for (int p = 0; p < P; p++) on = on || base[(static_cast<size_t>(p) * m3 + v) * dk::RB] != 0.f;
-                if (on) mk |= tc1_voxel_stages(v / (m * m), (v / m) % m, v % m, m);
-            }
+            if (pos < n_slots) mk |= masks[perm ? perm[pos] : pos];
         }
-    } else {
+    } else if (threadIdx.x == 0) {
         mk = nstg >= 64 ? ~0ull : (1ull << nstg) - 1ull;
     }
-    atomicOr(&s_mk, mk);
+    __shared__ unsigned long long s_mk[4];
+    const unsigned lo = __reduce_or_sync(0xffffffffu, static_cast<unsigned>(mk));
+    const unsigned hi = __reduce_or_sync(0xffffffffu, static_cast<unsigned>(mk >> 32));
+    if (lane == 0) s_mk[threadIdx.x >> 5] = (static_cast<unsigned long long>(hi) << 32) | lo;
     __syncthreads();
     if (threadIdx.x != 0) return;
-    mk = s_mk;
+    mk = s_mk[0] | s_mk[1] | s_mk[2] | s_mk[3];
     if (mk == 0ull) mk = 1ull;   // all-zero block: one zero-weight stage writes the accumulators
     int i = 0;
     for (int st = 0; st < nstg; st++)
         if ((mk >> st) & 1ull) src[i++] = static_cast<uint16_t>(st);
     kinfo[blk] = make_int4(i, 0, static_cast<int>(static_cast<uint32_t>(mk)), static_cast<int>(static_cast<uint32_t>(mk >> 32)));
     if (ksum) atomicAdd(ksum, static_cast<unsigned>(i * KSTEPS));
+}
+
+// Segment boundaries of the dynamic tile scheduler (one CTA): the chunk space (block-major, cpb chunks per
+// block) is cut into ns contiguous segments of equal estimated cost, a chunk of block b costing (its ring
+// stages + e_cost) -- the occupancy schedule makes blocks' tiles differ in length, and segments of equal chunk
+// counts would leave CTAs with cheap blocks helping others (each help restarts top-k lists: bursts of
+// insertions).  seg[j] = first chunk of segment j, seg[ns] = n_blocks * cpb.
+__global__ void k_tc_segments(const int4* __restrict__ kinfo, int n_blocks, int cpb, int ns, int e_cost,
+                              long long* __restrict__ pref, long long* __restrict__ seg)
+{
+    __shared__ long long s_carry;
+    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+    __shared__ long long s_w[32];
+    if (threadIdx.x == 0) s_carry = 0;
+    __syncthreads();
+    // pref[b] = cost of the chunks of blocks [0, b)
+    for (int b0 = 0; b0 < n_blocks; b0 += blockDim.x) {
+        const int b = b0 + threadIdx.x;
+        long long c = b < n_blocks ? static_cast<long long>(cpb) * (kinfo[b].x + e_cost) : 0;
+        long long incl = c;
+        for (int d = 1; d < 32; d <<= 1) {
+            const long long t = __shfl_up_sync(0xffffffffu, incl, d);
+            if (lane >= d) incl += t;
+        }
+        if (lane == 31) s_w[warp] = incl;
+        __syncthreads();
+        long long wbase = 0;
+        for (int w = 0; w < warp; w++) wbase += s_w[w];
+        if (b < n_blocks) pref[b] = s_carry + wbase + incl - c;
+        __syncthreads();
+        if (threadIdx.x == blockDim.x - 1) s_carry += wbase + incl;
+        __syncthreads();
+    }
+    const long long total = s_carry;
+    for (int j = threadIdx.x; j <= ns; j += blockDim.x) {
+        long long c;
+        if (j == ns) {
+            c = static_cast<long long>(n_blocks) * cpb;
+        } else {
+            const long long t = total * j / ns;
+            int lo = 0, hi = n_blocks - 1;   // last block with pref <= t
+            while (lo < hi) {
+                const int mid = (lo + hi + 1) >> 1;
+                if (pref[mid] <= t) lo = mid;
+                else hi = mid - 1;
+            }
+            const long long w = kinfo[lo].x + e_cost;
+            c = static_cast<long long>(lo) * cpb + min(static_cast<long long>(cpb), (t - pref[lo]) / w);
+        }
+        seg[j] = c;
+    }
 }
 
 // Variant 1 A operand, compacted: entry i of block b = dense K-step ksrc[b][i] of the units at the block's
