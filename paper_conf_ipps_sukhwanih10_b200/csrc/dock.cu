@@ -39,6 +39,8 @@ struct DevBuf {
 struct TcPlan {                // per-(variant, probe size) plan of the tcgen05 engine
     bool ok = false;
     CUtensorMap tmap, tmap_pair;   // (hi,lo) receptor copy and PAIR copy (Rhi(x), Rhi(x+1))
+    CUtensorMap tmap_b;            // variant 1: main half-box B (z planes [mh, m)); variant 1's tmap covers [0, mh)
+    int box_bytes_b = 0, rec_off_b = 0;
     int ntt = 0, q = 0, ntx = 0, nty = 0, ntiles = 0;   // translations per row, rows per tile, tile counts
     int S1 = 0, S1p = 0, S2 = 0, S2p = 0;                // variant 1: pass-1 / pass-2 K-steps (real, padded)
     int box_bytes = 0, box_bytes_pair = 0, rec_stage_bytes = 0, n_rec_stages = 0, smem = 0, nsteps = 0, wstages = 0;
@@ -366,9 +368,14 @@ dock_status make_tc_plan(dock_ctx* ctx, int m, int v)
         pl.TXBP = tc::pair_box_txb(m);
         TYB = pl.q + m - 1;
         TZB = m;
-        pl.box_bytes = 16 * TXB * TYB * TZB;
+        // the main box as two half-boxes (z planes [0, mh) and [mh, m)) with their own barriers: the next tile's
+        // half A streams in while this tile still reads half B and the pair box (dock_tc.cuh: k_corr_tc)
+        const int mh = (m + 1) / 2;
+        pl.box_bytes = 16 * TXB * TYB * mh;
+        pl.box_bytes_b = 16 * TXB * TYB * (m - mh);
+        pl.rec_off_b = round_up(pl.box_bytes, 128);
         pl.box_bytes_pair = 16 * pl.TXBP * TYB * TZB;
-        pl.rec_stage_bytes = round_up(pl.box_bytes, 128);   // offset of the pair box
+        pl.rec_stage_bytes = round_up(pl.rec_off_b + pl.box_bytes_b, 128);   // offset of the pair box
         rec_bytes = pl.rec_stage_bytes + round_up(pl.box_bytes_pair, 128);
         pl.n_rec_stages = 2;   // main box + pair box
         const int MXP = (m + 1) / 2, MXQ = (m + 3) / 4;
@@ -406,10 +413,16 @@ dock_status make_tc_plan(dock_ctx* ctx, int m, int v)
     cuuint64_t dims[5] = {8, X, Y, Z, (cuuint64_t)ctx->tc_Gch};
     cuuint64_t strides[4] = {16, X * 16, X * Y * 16, X * Y * Z * 16};
     cuuint32_t es[5] = {1, 1, 1, 1, 1};
-    for (int which = 0; which < 2; which++) {
-        cuuint32_t box[5] = {8, (cuuint32_t)(which && v == 1 ? pl.TXBP : TXB), (cuuint32_t)TYB, (cuuint32_t)TZB, 1};
-        CUresult r = fn(which ? &pl.tmap_pair : &pl.tmap, CU_TENSOR_MAP_DATA_TYPE_BFLOAT16, 5,
-                        which ? (void*)ctx->d_rec_pair : (void*)ctx->d_rec_tc, dims, strides, box, es,
+    for (int which = 0; which < 3; which++) {
+        const int mh = (m + 1) / 2;
+        if (which == 2 && (v != 1 || m - mh == 0 || m - mh == mh)) {
+            pl.tmap_b = pl.tmap;   // same half-box shape (or no second half)
+            continue;
+        }
+        const int tzb = v != 1 ? TZB : which == 0 ? mh : which == 2 ? m - mh : TZB;
+        cuuint32_t box[5] = {8, (cuuint32_t)(which == 1 && v == 1 ? pl.TXBP : TXB), (cuuint32_t)TYB, (cuuint32_t)tzb, 1};
+        CUresult r = fn(which == 1 ? &pl.tmap_pair : which == 2 ? &pl.tmap_b : &pl.tmap, CU_TENSOR_MAP_DATA_TYPE_BFLOAT16, 5,
+                        which == 1 ? (void*)ctx->d_rec_pair : (void*)ctx->d_rec_tc, dims, strides, box, es,
                         CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_L2_256B,
                         CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
         if (r != CUDA_SUCCESS) return fail(ctx, DOCK_E_CUDA, "cuTensorMapEncodeTiled (bf16) failed (%d)", (int)r);
@@ -420,7 +433,7 @@ dock_status make_tc_plan(dock_ctx* ctx, int m, int v)
 
 cudaError_t launch_tc(int m, int v, bool grid, const TcPlan& pl, const tc::TcArgs& a, int nblocks, cudaStream_t st)
 {
-    if (v == 1) return dock_launch_tc1(m, grid, pl.tmap, pl.tmap_pair, pl.smem, a, nblocks, st);
+    if (v == 1) return dock_launch_tc1(m, grid, pl.tmap, pl.tmap_pair, pl.tmap_b, pl.smem, a, nblocks, st);
     return dock_launch_tcs(m, pl.ntt, grid, pl.tmap, pl.tmap_pair, pl.smem, a, nblocks, st);
 }
 
@@ -678,6 +691,8 @@ tc::TcArgs tc_args(dock_ctx* ctx, int m, int v, int n_slots, int G, const unsign
     }
     a.box_bytes = tp.box_bytes;
     a.box_bytes_pair = tp.box_bytes_pair;
+    a.box_bytes_b = tp.box_bytes_b;
+    a.rec_off_b = tp.rec_off_b;
     a.rec_stage_bytes = tp.rec_stage_bytes;
     a.n_rec_stages = tp.n_rec_stages;
     a.wstages = tp.wstages;

@@ -13,8 +13,8 @@
 cudaError_t dock_launch_ffma(int m, bool grid, const CUtensorMap& tmap, int smem, const dk::CorrArgs& a, int nblocks,
                              cudaStream_t st);
 // tcgen05 variant 1 k_corr_tc<m, grid> (one channel group, resident boxes, NTT = 128, Q = 4)
-cudaError_t dock_launch_tc1(int m, bool grid, const CUtensorMap& tmap, const CUtensorMap& tmap_pair, int smem,
-                            const tc::TcArgs& a, int nblocks, cudaStream_t st);
+cudaError_t dock_launch_tc1(int m, bool grid, const CUtensorMap& tmap, const CUtensorMap& tmap_pair,
+                            const CUtensorMap& tmap_b, int smem, const tc::TcArgs& a, int nblocks, cudaStream_t st);
 // tcgen05 variant 2 k_corr_tcs<m, ntt, q(ntt), grid> (streamed planes); ntt in {64, 128, 160}
 cudaError_t dock_launch_tcs64(int m, bool grid, const CUtensorMap& tmap, const CUtensorMap& tmap_pair, int smem,
                               const tc::TcArgs& a, int nblocks, cudaStream_t st);

@@ -72,6 +72,8 @@ struct TcArgs {
                                 // blocks' schedule lengths (k_tc_segments); nullptr = equal chunk counts
     int box_bytes;              // bytes of one receptor TMA box (variant 1: the main box; variant 2: one z-plane)
     int box_bytes_pair;         // variant 1: bytes of the pair box
+    int box_bytes_b, rec_off_b; // variant 1: the main box is two half-boxes, z planes [0, mh) at 0 (box_bytes) and
+                                // [mh, m) at rec_off_b (box_bytes_b, 0 when m = 1), each with its own barriers
     int rec_stage_bytes;        // variant 1: offset of the pair box; variant 2: one receptor ring slot (unit)
     int n_rec_stages;           // variant 2: receptor ring depth (units)
     int wstages;                // weight ring depth (3..WSTAGES)
@@ -437,7 +439,8 @@ __host__ __device__ constexpr uint32_t pair_off2(int m, int s, uint32_t row16, u
 // stream holds only the block's active stages.  The schedule stays fully unrolled (immediate receptor offsets).
 template <int M, bool GRID>
 __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__ CUtensorMap tmap,
-                                                          const __grid_constant__ CUtensorMap tmap_pair, const TcArgs a)
+                                                          const __grid_constant__ CUtensorMap tmap_pair,
+                                                          const __grid_constant__ CUtensorMap tmap_b, const TcArgs a)
 {
     constexpr int Q = 4;
     constexpr int KS = KSTEPS;                 // K-steps per weight-ring stage (one wait/commit per KS steps)
@@ -450,16 +453,22 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
     constexpr uint32_t ROWTY = static_cast<uint32_t>(Q + M - 1) * ROW16;
     constexpr uint32_t ROW16P = static_cast<uint32_t>(pair_box_txb(M)) * 16u;   // pair box row pitch
     constexpr uint32_t ROWTYP = static_cast<uint32_t>(Q + M - 1) * ROW16P;
+    // main half-boxes: A = z planes [0, MH) at 0, B = [MH, M) at OFFB (128-B aligned for TMA); pass-1 K-steps
+    // from KB on read B, so B is needed from stage SB on and A is done after stage SA
+    constexpr int MH = (M + 1) / 2;
+    constexpr uint32_t OFFB = (MH * ROWTY + 127u) / 128u * 128u, GAPB = OFFB - MH * ROWTY;
+    constexpr int KB = MH * MXP * M, SB = KB / KS, SA = (KB - 1) / KS;
+    constexpr bool HAS_B = M > MH;
     static_assert(Q * NT <= 512, "TMEM has 512 columns");
     extern __shared__ __align__(128) unsigned char smem[];   // TMA destinations: 128 B; no-swizzle UMMA operands: 16 B
     constexpr int NCR = 4;                     // chunk ring: the weight producer posts, the other roles take
-    __shared__ uint64_t bars[2 * 2 + 2 * WSTAGES + 2 * Q + 2 * NCR];
+    __shared__ uint64_t bars[2 * 3 + 2 * WSTAGES + 2 * Q + 2 * NCR];
     __shared__ uint32_t tmem_base_s;
     __shared__ long long s_cg[NCR];            // chunk: first (block, tile) pair g = block * ntiles + tile
     __shared__ int s_cn[NCR];                  // chunk: tiles (0 = no more work)
-    uint64_t* rec_full = bars;
-    uint64_t* rec_empty = bars + 2;
-    uint64_t* w_full = bars + 4;
+    uint64_t* rec_full = bars;        // [3]: main half-box A, pair box, main half-box B
+    uint64_t* rec_empty = bars + 3;
+    uint64_t* w_full = bars + 6;
     uint64_t* w_empty = w_full + WSTAGES;
     uint64_t* tm_full = w_empty + WSTAGES;   // [Q]: row q accumulated (the staircase finishes rows one by one)
     uint64_t* tm_empty = tm_full + Q;        // [Q]: row q drained, so the next tile restarts row by row
@@ -504,7 +513,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
     unsigned char* w_smem = smem + a.rec_stage_bytes + ((a.box_bytes_pair + 127) & ~127);
 
     if (threadIdx.x == 0) {
-        for (int i = 0; i < 2; i++) {
+        for (int i = 0; i < 3; i++) {
             dk::mbar_init(&rec_full[i], 1);
             dk::mbar_init(&rec_empty[i], 1);
         }
@@ -659,17 +668,24 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
             if (elect_one()) {
                 dk::prefetch_tmap(&tmap);
                 dk::prefetch_tmap(&tmap_pair);
+                dk::prefetch_tmap(&tmap_b);
                 int ti = 0;   // tiles so far (buffer phases)
                 long long g;
                 for (int n; (n = take_chunk(g, true)) > 0;) {
                     const int t0 = static_cast<int>(g % a.ntiles);
                     int tx = t0 % a.ntx, ty = (t0 / a.ntx) % a.nty, tz = t0 / (a.ntx * a.nty);
                     for (int j = 0; j < n; j++, ti++) {
-                        for (int which = 0; which < 2; which++) {
+                        // in the order the MMAs need them: half-box A, half-box B, pair box
+                        for (int k = 0; k < 3; k++) {
+                            const int which = k == 0 ? 0 : k == 1 ? 2 : 1;
+                            if (which == 2 && !HAS_B) continue;
                             if (ti > 0) twait(&rec_empty[which], (ti - 1) & 1, tr, tw1);
-                            dk::mbar_arrive_expect_tx(&rec_full[which], which ? a.box_bytes_pair : a.box_bytes);
-                            tma_load_5d(rec_smem + which * a.rec_stage_bytes, which ? &tmap_pair : &tmap, 0,
-                                        tx * NT, ty * Q, tz, 0, &rec_full[which]);
+                            dk::mbar_arrive_expect_tx(&rec_full[which], which == 0   ? a.box_bytes
+                                                                        : which == 2 ? a.box_bytes_b
+                                                                                     : a.box_bytes_pair);
+                            tma_load_5d(rec_smem + (which == 0 ? 0 : which == 2 ? a.rec_off_b : a.rec_stage_bytes),
+                                        which == 0 ? &tmap : which == 2 ? &tmap_b : &tmap_pair, 0, tx * NT, ty * Q,
+                                        tz + (which == 2 ? MH : 0), 0, &rec_full[which]);
                         }
                         if (++tx == a.ntx) {
                             tx = 0;
@@ -702,6 +718,11 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
             const uint64_t dA0 = umma_desc(w0, ROT * 16, 128);                 // + (slot offset >> 4)
             const uint64_t dB0 = umma_desc(rec0, 16, 128);                     // + (voxel offset >> 4)
             const uint64_t dP0 = umma_desc(rec0 + a.rec_stage_bytes, 32, 128);
+            // byte offset of pass-1 K-step s: z planes from MH on sit in half-box B, GAPB further on
+            constexpr auto off1 = [](int s) constexpr -> uint32_t {
+                const int t = s < S1 ? s : S1 - 1;
+                return pair_off1(M, s, ROW16, ROWTY) + (t / (MXP * M) >= MH ? GAPB : 0u);
+            };
             if (elect_one()) {
                 uint32_t ws = 0, wph = 0;   // ring slot / phase of the next stage
                 const uint32_t nws = static_cast<uint32_t>(a.wstages);
@@ -747,6 +768,10 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                 for (int j = 0; j < n; j++, ti++) {
                     twait(&rec_full[0], ti & 1, tr, tw2);
                     tc_fence_after();
+                    if constexpr (HAS_B && SB < D) {   // the head reads half-box B too
+                        twait(&rec_full[2], ti & 1, tr, tw2);
+                        tc_fence_after();
+                    }
                     // pass 1, stages [0, D): row by row, each row after the epilogue released it
 #pragma unroll
                     for (int q = 0; q < Q; q++) {
@@ -768,7 +793,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
 #pragma unroll
                             for (int ks = 0; ks < KS; ks++)
                                 umma_bf16(tmem + q * NT, da0 + ((ks * WCHUNK) >> 4),
-                                          dB0 + ((pair_off1(M, st * KS + ks, ROW16, ROWTY) + q * ROW16) >> 4), idesc,
+                                          dB0 + ((off1(st * KS + ks) + q * ROW16) >> 4), idesc,
                                           (rk == 0 && ks == 0) ? 0u : 1u);
                         }
                     }
@@ -777,11 +802,19 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                         umma_commit(&w_empty[slot_of(i, ph)]);
                     }
                     advance(nh);
+                    if constexpr (SA < D) umma_commit(&rec_empty[0]);   // half-box A done with the head
                     int nact = nh;   // active stages issued so far in this tile (0: the next one overwrites)
                     // pass 1, stages [D, NS1): all rows per stage
 #pragma unroll
                     for (int st = D; st < NS1; st++) {
-                        if (!act(st)) continue;
+                        if (HAS_B && SB >= D && st == SB) {   // the first stage that reads half-box B
+                            twait(&rec_full[2], ti & 1, tr, tw2);
+                            tc_fence_after();
+                        }
+                        if (!act(st)) {
+                            if (SA >= D && st == SA) umma_commit(&rec_empty[0]);
+                            continue;
+                        }
                         twait(&w_full[ws], wph, tr, tw1);
                         tc_fence_after();
                         const uint64_t da0 = dA0 + ((ws * STAGE) >> 4);
@@ -791,13 +824,14 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
 #pragma unroll
                             for (int q = 0; q < Q; q++)
                                 umma_bf16(tmem + q * NT, da0 + ((ks * WCHUNK) >> 4),
-                                          dB0 + ((pair_off1(M, st * KS + ks, ROW16, ROWTY) + q * ROW16) >> 4), idesc,
+                                          dB0 + ((off1(st * KS + ks) + q * ROW16) >> 4), idesc,
                                           ks == 0 ? acc0 : 1u);
                         umma_commit(&w_empty[ws]);
                         advance(1);
                         nact++;
+                        if (SA >= D && st == SA) umma_commit(&rec_empty[0]);   // half-box A done
                     }
-                    umma_commit(&rec_empty[0]);
+                    if constexpr (HAS_B) umma_commit(&rec_empty[2]);
                     twait(&rec_full[1], ti & 1, tr, tw2);
                     tc_fence_after();
                     // pass 2, stages [0, NS2 - D): all rows per stage
