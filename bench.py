@@ -302,7 +302,10 @@ def run_ours(args):
 
     c, k, R, w, probes, rot, desc = workload(args.config, args.k, args.rho, args.rotations)
     n_units = c.n_probes * c.n_rot
-    b, e = parallel.shard_range(n_units, rank, world)
+    # rotation sharding: this rank docks every probe over its contiguous rotation slice [r0, r1) (units
+    # probe-major within the slice); world == 1: the whole unit range
+    r0, r1 = parallel.shard_range(c.n_rot, rank, world)
+    b, e = 0, c.n_probes * (r1 - r0)
     ctx = D.dock_init(torch.from_numpy(R).to(dev), torch.from_numpy(w).to(dev), g.SPACING, m_max=c.m,
                       device=local)
     if args.regions:
@@ -318,8 +321,22 @@ def run_ours(args):
     # probe descriptors marshalled once (the probe arrays stay where they are: device here, host in e2e)
     probes_dev = D.dock_probes(ctx, probes_dev)
     rot_dev = torch.from_numpy(rot).to(dev)
+    shard_mode = "single GPU"
     if world > 1:
-        pg = parallel.pose_gather(n_units, k, dev)   # preallocated all-gather buffer; poses land in its slot
+        # block sharding (tcgen05 variant 1: every rank clusters all units, docks its blocks of the common block
+        # order, one NCCL all-reduce MAX combines) when the engine allows it, else rotation sharding + all-gather
+        try:
+            parallel.dock_probe_sharded_blocks(ctx, probes_dev, rot_dev, k, args.rho, sync=True)
+            shard_mode = "blocks"
+        except D.DockError:
+            shard_mode = "rotations"
+    if shard_mode == "blocks":
+        bb = parallel.block_shard_buffer(n_units, k, dev)
+        r0, r1, b, e = 0, c.n_rot, 0, n_units
+        pg = None
+        out = bb.buf
+    elif world > 1:
+        pg = parallel.rotation_gather(c.n_probes, c.n_rot, k, dev)   # preallocated all-gather; poses land in its slot
         out = pg.slot
     else:
         pg = None
@@ -330,8 +347,11 @@ def run_ours(args):
 
     def step():
         # asynchronous: device output, no host sync inside the step (errors surface at dock_sync below)
+        if shard_mode == "blocks":
+            parallel.dock_probe_sharded_blocks(ctx, probes_dev, rot_dev, k, args.rho, sync=False)
+            return
         if e > b:
-            D.dock_probe_batch(ctx, probes_dev, rot_dev, b, e, k, args.rho, out=out)
+            D.dock_probe_batch(ctx, probes_dev, rot_dev[r0:r1], b, e, k, args.rho, out=out)
         if world > 1:
             pg.gather()
 
@@ -391,16 +411,19 @@ def run_ours(args):
     # ---- e2e through the public API with host buffers (H2D of inputs + D2H of poses inside)
     e2e = None
     if not args.no_e2e:
-        h2d = rot.nbytes + sum(p.xyz.nbytes + p.coef.nbytes for p in probes) + 4 * (len(probes) + 1)
+        h2d = rot[r0:r1].nbytes + sum(p.xyz.nbytes + p.coef.nbytes for p in probes) + 4 * (len(probes) + 1)
         d2h = n_units * k * 16
-        out2 = pg.slot if world > 1 else torch.empty((e - b, k, 4), dtype=torch.int32, device=dev)
+        out2 = pg.slot if pg is not None else torch.empty((e - b, k, 4), dtype=torch.int32, device=dev)
         probes_host = D.dock_probes(ctx, probes)   # host arrays: staged and copied H2D inside every call
 
         def step_e2e():
             # host numpy inputs (pinned staging + H2D inside the call), device poses, D2H read of the result
-            if e > b:
-                D.dock_probe_batch(ctx, probes_host, rot, b, e, k, args.rho, out=out2)
-            full = pg.gather() if world > 1 else out2
+            if shard_mode == "blocks":
+                full = parallel.dock_probe_sharded_blocks(ctx, probes_host, rot, k, args.rho, sync=False)
+            else:
+                if e > b:
+                    D.dock_probe_batch(ctx, probes_host, rot[r0:r1], b, e, k, args.rho, out=out2)
+                full = pg.gather() if world > 1 else out2
             if rank == 0:
                 full.cpu()
 
@@ -425,6 +448,9 @@ def run_ours(args):
     pk, pk_kind = peaks()
     info = D.dock_get_info(ctx)
     units_local = e - b
+    if shard_mode == "blocks":   # this rank's blocks rank, rank + world, ... of 128 units
+        nb = -(-n_units // 128)
+        units_local = sum(min(128, n_units - bb_ * 128) for bb_ in range(rank, nb, world))
     flops_launch = 2.0 * c.P * c.m ** 3 * c.n[0] * c.n[1] * c.n[2] * units_local   # algorithmic (dense) FLOPs
     corr_ms = corr_max / args.steps
     roof = roofline(pk, pk_kind, info, c, flops_launch, corr_ms, ms_step, units_local)
@@ -484,7 +510,8 @@ def run_ours(args):
 
     if rank == 0:
         desc = dict(desc)
-        desc.update({"parallelism": f"rotation-shard x{world}" if world > 1 else "single GPU",
+        desc.update({"parallelism": (f"{'block' if shard_mode == 'blocks' else 'rotation'}-shard x{world}"
+                                     if world > 1 else "single GPU"),
                      "l2": f"flushed between timed steps ({flush.numel() * 4 >> 20} MiB write); "
                            f"receptor {R.nbytes >> 20} MiB fits in L2",
                      "regions": info["regions_last"], "items": info["items_last"], "engine": roof["engine"],

@@ -179,14 +179,22 @@ typedef enum {
                                      above the compiled maximum are clamped to it) */
     DOCK_TUNE_TC_CHUNK = 7,       /* tcgen05 variant 1: tiles per dynamically scheduled chunk (0 = auto, 4;
                                      1..4096); one persistent CTA per SM takes chunks from a device counter */
-    DOCK_TUNE_TC_SCHEDULE = 8     /* tcgen05 variant 1 K-step schedule.  A K-step (16 products per accumulator) whose
-                                     probe weights are zero for all 128 rotations of a block adds exact zeros, so a
-                                     block runs only its occupied K-steps (a probe grid has at most one occupied voxel
-                                     per atom).  0 (default): occupancy schedule, and for m <= 4 the
-                                     units are first grouped into blocks with few distinct occupied K-steps (greedy,
-                                     on the device); 1: occupancy schedule over blocks of consecutive units; 2: dense
-                                     (every K-step).  Scores are bitwise identical in all three modes (skipped
-                                     products are exact zeros). */
+    DOCK_TUNE_TC_SCHEDULE = 8,    /* tcgen05 variant 1 schedule.  A ring stage (4 K-steps of 16 products per accumulator)
+                                     whose probe weights are zero for all 128 rotations of a block adds exact zeros, so a
+                                     block runs only its active stages (a probe grid has at most one occupied voxel per
+                                     atom).  0 (default): occupancy schedule, the units first grouped into
+                                     blocks with few distinct active stages (greedy, on the device, deterministic); 1:
+                                     occupancy schedule over blocks of consecutive units; 2: dense (every stage).  Scores
+                                     are bitwise identical in all three modes (skipped products are exact zeros). */
+    DOCK_TUNE_SHARD = 9           /* block sharding for multi-GPU runs: value = world << 16 | rank (world 1 = off).  With
+                                     world > 1, dock_probe_batch docks only the rotation blocks rank, rank + world, ...
+                                     of the call's (clustered, deterministic) block order -- every rank clusters the
+                                     whole unit range, so the blocks stay as good as on one GPU -- and writes only its
+                                     units' rows of `out` (a DEVICE buffer: host output copies every row back); the caller
+                                     pre-fills `out` with 0x80000000 in every field and
+                                     combines the ranks' buffers with an elementwise int32 MAX (every field of a written
+                                     row is > INT32_MIN except the bits of a -0.0 score, which MAX keeps).  Needs the
+                                     tcgen05 variant-1 engine (DOCK_E_UNSUPPORTED otherwise). */
 } dock_tune_key;
 
 dock_status dock_set_tuning(dock_ctx* ctx, int key, int64_t value);

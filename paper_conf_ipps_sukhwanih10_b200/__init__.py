@@ -12,7 +12,7 @@ from .dock import (  # noqa: F401
 )
 from ._native import (  # noqa: F401
     DOCK_MAX_K, DOCK_MAX_M, DOCK_MAX_TERMS, DOCK_POSE_FALLBACK, DOCK_TUNE_CAND_CAP, DOCK_TUNE_ENGINE, DOCK_TUNE_TC_VARIANT, DOCK_TUNE_TC_CHUNK,
-    DOCK_TUNE_TC_SCHEDULE,
+    DOCK_TUNE_TC_SCHEDULE, DOCK_TUNE_SHARD,
     DOCK_TUNE_FORCE_FALLBACK, DOCK_TUNE_REGIONS, EXPORTS, LIB_PATH,
 )
 from . import parallel  # noqa: F401,E402

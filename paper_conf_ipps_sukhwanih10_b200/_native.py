@@ -26,6 +26,7 @@ DOCK_TUNE_TC_VARIANT = 5
 DOCK_TUNE_TC_EPILOGUE_WARPS = 6
 DOCK_TUNE_TC_CHUNK = 7
 DOCK_TUNE_TC_SCHEDULE = 8
+DOCK_TUNE_SHARD = 9
 DOCK_ENGINE_AUTO, DOCK_ENGINE_FFMA, DOCK_ENGINE_TC, DOCK_ENGINE_FFT, DOCK_ENGINE_SPARSE = 0, 1, 2, 3, 4
 
 STATUS_NAMES = {0: "DOCK_OK", -1: "DOCK_E_INVALID_ARG", -2: "DOCK_E_UNSUPPORTED",

@@ -104,6 +104,9 @@ struct dock_ctx {
     // variant 1 occupancy schedule of the main pass / of the fallback: K-step tables, source steps, per-block
     // (stages, first pair entry), clustering permutation and unit masks
     DevBuf tc_ksrc, tc_kinfo, tc_perm, tc_umask, tc_sorted, fb_ksrc, fb_kinfo, fb_umask, tc_seg, tc_pref;
+    int shard_rank = 0, shard_world = 1;   // DOCK_TUNE_SHARD: block sharding of the variant-1 block order
+    int tc_nblk_local = -1;    // blocks of the last main pass this rank docks (-1: all)
+    DevBuf tc_blkmap, tc_owned;
     int tc_seg_cost = 8;       // per-tile cost of a chunk beyond its ring stages, in ring stages (prod: 0 / 3 / 6 /
                                // 9 / 12 / 24 -> 12.20 / 11.79 / 11.40 / 11.35 / 11.48 / 11.84 ms); DOCK_TC_SEG_COST
                                // (environment) overrides it
@@ -688,6 +691,10 @@ tc::TcArgs tc_args(dock_ctx* ctx, int m, int v, int n_slots, int G, const unsign
         const bool fb = W == static_cast<const unsigned char*>(ctx->fb_W.p);
         a.kinfo = static_cast<const int4*>(fb ? ctx->fb_kinfo.p : ctx->tc_kinfo.p);
         a.perm = (!fb && ctx->tc_perm_on) ? static_cast<const int*>(ctx->tc_perm.p) : nullptr;
+        if (!fb && ctx->tc_nblk_local >= 0) {   // block sharding
+            a.blkmap = static_cast<const int*>(ctx->tc_blkmap.p);
+            a.n_blocks = ctx->tc_nblk_local;
+        }
     }
     a.box_bytes = tp.box_bytes;
     a.box_bytes_pair = tp.box_bytes_pair;
@@ -712,7 +719,7 @@ tc::TcArgs tc_args(dock_ctx* ctx, int m, int v, int n_slots, int G, const unsign
 // CTAs of a tensor-core launch over n_slots rotations.
 int64_t tc_ctas(const tc::TcArgs& a, int n_slots, int n_sms)
 {
-    const int64_t n_blocks = (n_slots + tc::ROT - 1) / tc::ROT;
+    const int64_t n_blocks = a.blkmap ? a.n_blocks : (n_slots + tc::ROT - 1) / tc::ROT;
     if (a.chunk > 0) return std::min<int64_t>(n_sms, n_blocks * ((a.ntiles + a.chunk - 1) / a.chunk));
     return n_blocks * a.G;
 }
@@ -1003,7 +1010,7 @@ sp::SpArgs sp_args(dock_ctx* ctx, const SpCall& sc, const sp::Group* d_groups, i
 // DOCK_TUNE_TC_SCHEDULE 0), then per block the table of occupied K-steps, then the A operand in table order.
 // fb: the fallback's buffers (no clustering; n_live = the live count of the device-driven loop).
 dock_status pack_weights_tc(dock_ctx* ctx, int m, int v, int n_slots, const float* Lw, bool fb = false,
-                            const unsigned* n_live = nullptr)
+                            const unsigned* n_live = nullptr, bool shard = false)
 {
     const TcPlan& tp = ctx->tcplan[v][m];
     const int64_t n_blocks = (n_slots + tc::ROT - 1) / tc::ROT;
@@ -1047,7 +1054,22 @@ dock_status pack_weights_tc(dock_ctx* ctx, int m, int v, int n_slots, const floa
             ctx->kernels_last++;
             perm = static_cast<const int*>(ctx->tc_perm.p);
         }
-        if (!fb) ctx->tc_perm_on = perm != nullptr;
+        if (!fb) {
+            ctx->tc_perm_on = perm != nullptr;
+            ctx->tc_nblk_local = -1;
+            if (shard && ctx->shard_world > 1) {   // block sharding: this rank's blocks of the (clustered) block order
+                TRY(ensure(ctx, ctx->tc_blkmap, sizeof(int) * n_blocks));
+                TRY(ensure(ctx, ctx->tc_owned, (size_t)n_slots));
+                tc::k_tc_shard_blocks<<<(int)std::min<int64_t>((n_blocks * tc::ROT + 255) / 256, 4096), 256, 0,
+                                        ctx->stream>>>(perm, n_slots, (int)n_blocks, ctx->shard_rank, ctx->shard_world,
+                                                       static_cast<int*>(ctx->tc_blkmap.p),
+                                                       static_cast<unsigned char*>(ctx->tc_owned.p));
+                CU(cudaGetLastError());
+                ctx->kernels_last++;
+                ctx->tc_nblk_local =
+                    n_blocks > ctx->shard_rank ? (int)((n_blocks - ctx->shard_rank + ctx->shard_world - 1) / ctx->shard_world) : 0;
+            }
+        }
         tc::k_tc_block_tables<<<(int)n_blocks, 128, 0, ctx->stream>>>(
             um, perm, n_slots, tp.nsteps, static_cast<uint16_t*>(ks.p), static_cast<int4*>(ki.p),
             fb ? nullptr : reinterpret_cast<unsigned*>(ctx->d_small + 3));
@@ -1480,7 +1502,7 @@ void dock_destroy(dock_ctx* ctx)
                       &ctx->slots,   &ctx->units,    &ctx->Lw_fb,  &ctx->picks,    &ctx->fb_grid,  &ctx->fb_Lw,
                       &ctx->fb_W,    &ctx->fb_picks, &ctx->fb_slots, &ctx->fb_ctl,   &ctx->tc_ksrc,
                       &ctx->tc_kinfo, &ctx->tc_perm, &ctx->tc_umask, &ctx->tc_sorted, &ctx->fb_ksrc, &ctx->fb_kinfo,
-                      &ctx->fb_umask, &ctx->tc_seg,  &ctx->tc_pref};
+                      &ctx->fb_umask, &ctx->tc_seg,  &ctx->tc_pref, &ctx->tc_blkmap, &ctx->tc_owned};
     for (DevBuf* b : bufs)
         if (b->p) cudaFree(b->p);
     if (ctx->d_trace) cudaFree(ctx->d_trace);
@@ -1707,6 +1729,14 @@ dock_status dock_set_tuning(dock_ctx* ctx, int key, int64_t value)
             if (value < 0 || value > 4096) return fail(ctx, DOCK_E_INVALID_ARG, "tc chunk must be 0..4096");
             ctx->tc_chunk = (int)value;
             return DOCK_OK;
+        case DOCK_TUNE_SHARD: {
+            const int world = (int)(value >> 16), rank = (int)(value & 0xffff);
+            if (world < 1 || world > 4096 || rank >= world)
+                return fail(ctx, DOCK_E_INVALID_ARG, "shard: value = world << 16 | rank, 1 <= world, rank < world");
+            ctx->shard_world = world;
+            ctx->shard_rank = rank;
+            return DOCK_OK;
+        }
         case DOCK_TUNE_TC_SCHEDULE:
             if (value < 0 || value > 2) return fail(ctx, DOCK_E_INVALID_ARG, "tc schedule must be 0, 1 or 2");
             ctx->tc_sched = (int)value;
@@ -1832,6 +1862,8 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
         if (ctx->engine == 0 || ctx->engine == 4)
             TRY(sp_prepare(ctx, m, probes, n_probes, n_rot, unit_begin, unit_end, &sc));
         TRY(select_engine(ctx, m, sc.ok, sp_better(ctx, sc, m, n_units), &kind));
+        if (ctx->shard_world > 1 && kind != ENG_TC)
+            return fail(ctx, DOCK_E_UNSUPPORTED, "block sharding needs the tcgen05 variant-1 engine");
         TRY(fb_buffers(ctx, m, fb_chunk(ctx, kind), k));
     }
     const bool use_tc = kind == ENG_TC;
@@ -1902,8 +1934,10 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
         const int64_t n_blocks = (n_units + tc::ROT - 1) / tc::ROT;
         int v = 0, G = 0;
         if (!plan_tc_launch(ctx, m, n_units, &v, &G)) return fail(ctx, DOCK_E_UNSUPPORTED, "no tensor-core plan");
-        TRY(pack_weights_tc(ctx, m, v, n_units, static_cast<const float*>(ctx->Lw.p)));
+        TRY(pack_weights_tc(ctx, m, v, n_units, static_cast<const float*>(ctx->Lw.p), false, nullptr, true));
         ctx->tc_variant_last = v;
+        if (ctx->shard_world > 1 && v != 1)
+            return fail(ctx, DOCK_E_UNSUPPORTED, "block sharding needs the tcgen05 variant-1 engine");
         ctx->tc_ksteps_last = ctx->tcplan[v][m].nsteps;
         ctx->tc_m_last = m;
         tc::TcArgs ta = tc_args(ctx, m, v, n_units, G, static_cast<const unsigned char*>(ctx->Wtc.p));
@@ -1916,12 +1950,13 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
         ta.cand = candp;
         const int64_t items = tc_ctas(ta, n_units, ctx->n_sms);
         if (items > 0x7fffffff) return fail(ctx, DOCK_E_UNSUPPORTED, "too many work items");
-        if (v == 1 && ta.chunk > 0 && ctx->tc_sched != 2 && n_blocks <= (1 << 16)) {
+        if (v == 1 && ta.chunk > 0 && ctx->tc_sched != 2 && n_blocks <= (1 << 16) && items > 0) {
             // scheduler segments of equal estimated cost (blocks' occupancy schedules differ in length)
             TRY(ensure(ctx, ctx->tc_seg, sizeof(long long) * (items + 1)));
             TRY(ensure(ctx, ctx->tc_pref, sizeof(long long) * n_blocks));
             const int cpb = (ta.ntiles + ta.chunk - 1) / ta.chunk;
-            tc::k_tc_segments<<<1, 256, 0, ctx->stream>>>(ta.kinfo, (int)n_blocks, cpb, (int)items, ctx->tc_seg_cost,
+            tc::k_tc_segments<<<1, 256, 0, ctx->stream>>>(ta.kinfo, ta.blkmap, ta.blkmap ? ta.n_blocks : (int)n_blocks,
+                                                          cpb, (int)items, ctx->tc_seg_cost,
                                                           static_cast<long long*>(ctx->tc_pref.p),
                                                           static_cast<long long*>(ctx->tc_seg.p));
             CU(cudaGetLastError());
@@ -1930,7 +1965,7 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
         }
         if (ctx->d_trace) CU(cudaMemsetAsync(ctx->d_trace, 0, sizeof(unsigned long long) * tc::TR_N, ctx->stream));
         CU(cudaEventRecord(ctx->ev_corr[0], ctx->stream));
-        CU(launch_tc(m, v, false, ctx->tcplan[v][m], ta, (int)items, ctx->stream));
+        if (items > 0) CU(launch_tc(m, v, false, ctx->tcplan[v][m], ta, (int)items, ctx->stream));   // 0: no block here
         CU(cudaEventRecord(ctx->ev_corr[1], ctx->stream));
         if (ctx->d_trace) {
             std::vector<unsigned long long> hv(tc::TR_N);
@@ -2010,6 +2045,7 @@ dock_status dock_probe_batch(dock_ctx* ctx, const dock_probe_desc* probes, int n
     ma.fb_list = static_cast<int*>(ctx->fb_list.p);
     ma.fb_cnt = fb_cnt;
     ma.cand_max = cand_max;
+    ma.owned = (use_tc && ctx->tc_nblk_local >= 0) ? static_cast<const unsigned char*>(ctx->tc_owned.p) : nullptr;
     dk::k_merge<<<(n_units + 7) / 8, 256, 0, ctx->stream>>>(ma);
     CU(cudaGetLastError());
     ctx->kernels_last++;

@@ -572,6 +572,7 @@ struct MergeArgs {
     int* fb_list;              // flagged slots
     unsigned int* fb_cnt;
     unsigned int* cand_max;    // max candidate count seen (stats)
+    const unsigned char* owned;   // block sharding: units this rank docks (others: output rows untouched); nullptr = all
 };
 
 struct PoseOut {
@@ -595,6 +596,7 @@ __global__ void k_merge(MergeArgs a)
     const int wl = threadIdx.x >> 5, lane = threadIdx.x & 31;
     const int slot = blockIdx.x * (blockDim.x >> 5) + wl;
     if (slot >= a.n_slots) return;
+    if (a.owned && !a.owned[slot]) return;   // another rank's unit (block sharding)
     unsigned long long* picks = picks_s[wl];
     const unsigned int n_all = a.cnt[slot];
     const unsigned int n = min(n_all, static_cast<unsigned int>(a.cap));

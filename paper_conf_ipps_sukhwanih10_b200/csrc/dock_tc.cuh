@@ -68,6 +68,8 @@ struct TcArgs {
     const int4* kinfo;          // [block]: (ring stages of the compacted A stream, -, active K-step mask lo, hi)
     const int* perm;            // [block * ROT]: block position -> unit slot (occupancy clustering); nullptr =
                                 // identity
+    const int* blkmap;          // block sharding: [local block] -> block of the call's block order; nullptr = identity
+    int n_blocks;               // blocks this launch processes (local count under block sharding; 0 = all)
     const long long* seg;       // [gridDim.x + 1]: dynamic scheduler segment boundaries (chunk ids) balanced by the
                                 // blocks' schedule lengths (k_tc_segments); nullptr = equal chunk counts
     int box_bytes;              // bytes of one receptor TMA box (variant 1: the main box; variant 2: one z-plane)
@@ -477,7 +479,9 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
 
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     const int n_eff = a.n_live ? min(a.n_slots, static_cast<int>(*a.n_live)) : a.n_slots;
-    const long long live_blocks = (n_eff + ROT - 1) / ROT;
+    const long long live_blocks = a.n_blocks > 0 ? a.n_blocks : (n_eff + ROT - 1) / ROT;
+    // block of the call's block order for a local block index (block sharding: this rank's blocks only)
+    auto gblock = [&](long long lb) -> long long { return a.blkmap ? a.blkmap[lb] : lb; };
     // Work: a sequence of chunks (g, n) = n consecutive tiles of one rotation block starting at the (block,
     // tile) pair g = block * ntiles + tile.  Region mode: the one chunk (block, region) of this CTA.  Dynamic
     // mode: chunk c = (block c / cpb, tiles [(c % cpb) chunk, ..)), c in [0, n_chunks), split into NS
@@ -636,7 +640,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                 if (a.chunk > 0) c = fetch();   // one chunk of lookahead: the atomic hides behind the stream
                 n_tiles += n;
                 if (lane == 0) {
-                    const long long blk = g / a.ntiles;
+                    const long long blk = gblock(g / a.ntiles);
                     const unsigned char* wsrc = a.W + static_cast<size_t>(blk) * NSTEPS * WCHUNK;
                     const int nst = a.kinfo[blk].x;   // the block's active stages (compacted weight stream)
                     for (int ti = 0; ti < n; ti++) {
@@ -755,7 +759,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                     return MASKED ? __popcll(mk & ((1ull << (st & 63)) - 1ull)) : st;
                 };
                 for (int n; (n = take_chunk(g, true)) > 0;) {
-                    const long long blk = g / a.ntiles;
+                    const long long blk = gblock(g / a.ntiles);
                     if (MASKED && blk != mblk) {
                         const int4 inf = a.kinfo[blk];
                         smk = static_cast<unsigned long long>(static_cast<uint32_t>(inf.z)) |
@@ -927,7 +931,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                     th = __int_as_float(0x7f800000);
                     th_t = 0xffffffffu;
                     cur = blk;
-                    const int pos = static_cast<int>(blk) * ROT + r;   // position in the block order
+                    const int pos = static_cast<int>(gblock(blk)) * ROT + r;   // position in the block order
                     rot_ok = pos < n_eff;
                     slot = (a.perm && rot_ok) ? a.perm[pos] : pos;     // the unit it holds
                 }
@@ -1388,7 +1392,7 @@ __global__ void k_tc_unit_masks(const float* __restrict__ Lw, int n_slots, const
 }
 
 // Greedy grouping over distinct masks (stage masks of <= CB_BITS bits, one CTA per window of CL_W units): the
-// window's units are binned by mask (a counting sort); one warp then runs the greedy of
+// window's units are binned by mask (a stable counting sort); one warp then runs the greedy of
 // k_tc_cluster on the distinct masks -- a block takes every remaining mask already inside its union (all its
 // units, as far as the block has room), then all units of the mask that adds the fewest stages (ties: lowest
 // mask) -- and the take records are expanded into the permutation.  Same blocks as the unit greedy up to the
@@ -1455,11 +1459,24 @@ __global__ void __launch_bounds__(1024, 1) k_tc_cluster_bins(const unsigned long
             run += c;
         }
         if (lane == 31) s_nl = inz;
+        // stable counting sort: units in index order, 32 at a time (lanes with equal masks ranked by lane), so
+        // the permutation is a deterministic function of the masks (block sharding needs every rank to compute
+        // the same one)
+        __syncwarp();
+        for (int i0 = 0; i0 < n; i0 += 32) {
+            const int i = i0 + lane;
+            const int b = i < n ? static_cast<int>(S.umask[i]) : -1;
+            const unsigned grp = __match_any_sync(0xffffffffu, b);
+            const int rank = __popc(grp & ((1u << lane) - 1u));
+            const int at = i < n ? S.fill[b] + rank : 0;
+            __syncwarp();
+            if (i < n) {
+                srt[at] = w0 + i;
+                if (rank == 0) S.fill[b] += __popc(grp);
+            }
+            __syncwarp();
+        }
     }
-    __syncthreads();
-    // counting sort by mask (the order among units of equal masks is arbitrary: blocks, stage masks and every
-    // per-rotation result are the same for any order)
-    for (int i = tid; i < n; i += blockDim.x) srt[atomicAdd(&S.fill[S.umask[i]], 1)] = w0 + i;
     __syncthreads();
     if (warp == 0 && s_nl <= 32 * 8) {
         // the greedy over <= 256 distinct masks with the list in registers: lane L owns entries [8L, 8L + 8)
@@ -1774,8 +1791,8 @@ __global__ void k_tc_block_tables(const unsigned long long* __restrict__ masks, 
 // stages + e_cost) -- the occupancy schedule makes blocks' tiles differ in length, and segments of equal chunk
 // counts would leave CTAs with cheap blocks helping others (each help restarts top-k lists: bursts of
 // insertions).  seg[j] = first chunk of segment j, seg[ns] = n_blocks * cpb.
-__global__ void k_tc_segments(const int4* __restrict__ kinfo, int n_blocks, int cpb, int ns, int e_cost,
-                              long long* __restrict__ pref, long long* __restrict__ seg)
+__global__ void k_tc_segments(const int4* __restrict__ kinfo, const int* __restrict__ blkmap, int n_blocks, int cpb,
+                              int ns, int e_cost, long long* __restrict__ pref, long long* __restrict__ seg)
 {
     __shared__ long long s_carry;
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
@@ -1785,7 +1802,7 @@ __global__ void k_tc_segments(const int4* __restrict__ kinfo, int n_blocks, int 
     // pref[b] = cost of the chunks of blocks [0, b)
     for (int b0 = 0; b0 < n_blocks; b0 += blockDim.x) {
         const int b = b0 + threadIdx.x;
-        long long c = b < n_blocks ? static_cast<long long>(cpb) * (kinfo[b].x + e_cost) : 0;
+        long long c = b < n_blocks ? static_cast<long long>(cpb) * (kinfo[blkmap ? blkmap[b] : b].x + e_cost) : 0;
         long long incl = c;
         for (int d = 1; d < 32; d <<= 1) {
             const long long t = __shfl_up_sync(0xffffffffu, incl, d);
@@ -1813,10 +1830,23 @@ __global__ void k_tc_segments(const int4* __restrict__ kinfo, int n_blocks, int 
                 if (pref[mid] <= t) lo = mid;
                 else hi = mid - 1;
             }
-            const long long w = kinfo[lo].x + e_cost;
+            const long long w = kinfo[blkmap ? blkmap[lo] : lo].x + e_cost;
             c = static_cast<long long>(lo) * cpb + min(static_cast<long long>(cpb), (t - pref[lo]) / w);
         }
         seg[j] = c;
+    }
+}
+
+// Block sharding (multi-GPU): rank `rank` of `world` docks blocks b = rank, rank + world, ... of the call's block
+// order (interleaved, so every rank gets blocks from the whole cost range of the clustering); blkmap[lb] = its
+// lb-th block, owned[unit] = 1 for the units of those blocks.
+__global__ void k_tc_shard_blocks(const int* __restrict__ perm, int n_slots, int n_blocks, int rank, int world,
+                                  int* __restrict__ blkmap, unsigned char* __restrict__ owned)
+{
+    for (int pos = blockIdx.x * blockDim.x + threadIdx.x; pos < n_blocks * ROT; pos += gridDim.x * blockDim.x) {
+        const int b = pos / ROT;
+        if (pos % ROT == 0 && b % world == rank) blkmap[b / world] = b;
+        if (pos < n_slots) owned[perm ? perm[pos] : pos] = static_cast<unsigned char>(b % world == rank);
     }
 }
 

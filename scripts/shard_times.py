@@ -1,7 +1,9 @@
 #!/usr/bin/env python
 """Per-rank shard times of the multi-GPU rotation sharding, measured on ONE B200 (this sandbox has one GPU per
-call): for N in 1, 2, 4, 8 the unit block rank 0 would own (parallel.shard_range) is docked alone, steps
-enqueued back to back (the asynchronous path), CUDA-event timed.  The N-GPU step would add one NCCL
+call): for N in 1, 2, 4, 8 every rank's shard is docked alone, CUDA-event timed, and the projection takes the
+slowest rank.  Two shardings: "rotations" (every probe over the rank's rotation slice, parallel.dock_probe_sharded)
+and "blocks" (DOCK_TUNE_SHARD: every rank clusters all units and docks its blocks of the common block order,
+parallel.dock_probe_sharded_blocks; the collective is then one all-reduce MAX).  The N-GPU step would add one NCCL
 all-gather of N x 16 B x k x units/N poses (64 KB per rank at N = 8); it is NOT included.  The output is a
 projection input (per-rank work), not a multi-GPU measurement.   python scripts/shard_times.py [--config prod]"""
 import argparse
@@ -38,29 +40,58 @@ def main():
     probes = D.dock_probes(ctx, probes)   # descriptors marshalled once, as bench.py does
     n = c.n_probes * c.n_rot
     flush = torch.empty(64 << 20, dtype=torch.float32, device=dev)
-    res = {"config": args.config, "units": n, "note": __doc__.split("\n")[1].strip(), "per_n": {}}
-    for N in (1, 2, 4, 8):
-        b, e = parallel.shard_range(n, 0, N)
-        out = torch.empty((e - b, c.k, 4), dtype=torch.int32, device=dev)
+    res = {"config": args.config, "units": n, "note": "per-rank shard times on one B200 (see the docstring)"}
+    def timed(call):
         for _ in range(3):
-            D.dock_probe_batch(ctx, probes, rot, b, e, c.k, 1, out=out)
+            call()
         D.dock_sync(ctx)
         ts = []
         for i in range(args.steps):
             flush.fill_(float(i))
             e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
             e0.record()
-            D.dock_probe_batch(ctx, probes, rot, b, e, c.k, 1, out=out)
+            call()
             e1.record()
             e1.synchronize()
             ts.append(e0.elapsed_time(e1))
         D.dock_sync(ctx)
         info = D.dock_get_info(ctx)
-        res["per_n"][N] = {"units_rank0": e - b, "ms_median": statistics.median(ts), "ms_min": min(ts),
-                           "engine": info["engine_last"], "kernel_ms": info["corr_ms_last"]}
-    t1 = res["per_n"][1]["ms_median"]
-    for N, r in res["per_n"].items():
-        r["projected_efficiency_without_allgather"] = t1 / (N * r["ms_median"])
+        return statistics.median(ts), info["corr_ms_last"], info["engine_last"]
+
+    full = torch.empty((n, c.k, 4), dtype=torch.int32, device=dev)
+    for mode in ("rotations", "blocks"):
+        res[mode] = {}
+        for N in (1, 2, 4, 8):
+            ranks = []
+            for rk in range(N):
+                if mode == "rotations":   # every probe over this rank's rotation slice
+                    r0, r1 = parallel.shard_range(c.n_rot, rk, N)
+                    units = c.n_probes * (r1 - r0)
+                    out = torch.empty((units, c.k, 4), dtype=torch.int32, device=dev)
+                    rs = rot[r0:r1]
+                    ms, kms, eng = timed(lambda: D.dock_probe_batch(ctx, probes, rs, 0, units, c.k, 1, out=out))
+                    ranks.append({"rotations": [r0, r1], "units": units, "ms_median": ms, "kernel_ms": kms,
+                                  "engine": eng})
+                else:   # DOCK_TUNE_SHARD: all units clustered, this rank's blocks docked
+                    D.dock_set_tuning(ctx, D.DOCK_TUNE_SHARD, (N << 16) | rk)
+                    try:
+                        ms, kms, eng = timed(lambda: D.dock_probe_batch(ctx, probes, rot, 0, n, c.k, 1, out=full))
+                    except D.DockError as ex:
+                        ranks = None
+                        res[mode]["unsupported"] = str(ex)
+                        break
+                    finally:
+                        D.dock_set_tuning(ctx, D.DOCK_TUNE_SHARD, 1 << 16)
+                    ranks.append({"rank": rk, "ms_median": ms, "kernel_ms": kms, "engine": eng})
+            if ranks is None:
+                break
+            res[mode][N] = {"ranks": ranks, "ms_max_over_ranks": max(r["ms_median"] for r in ranks),
+                            "ms_mean_over_ranks": statistics.mean(r["ms_median"] for r in ranks)}
+        if 1 in res[mode]:
+            t1 = res[mode][1]["ms_max_over_ranks"]
+            for N, r in res[mode].items():
+                if isinstance(r, dict):
+                    r["projected_efficiency_without_collective"] = t1 / (N * r["ms_max_over_ranks"])
     print(json.dumps(res), flush=True)
     ctx.close()
 

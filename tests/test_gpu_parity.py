@@ -376,6 +376,36 @@ def test_tc_occupancy_schedule_integer_exact(D, orc):
         assert np.array_equal(poses["score"].astype(np.float64), s_o)
 
 
+@pytest.mark.parametrize("world", [2, 3, 8])
+def test_block_sharding_emulated_ranks(D, world):
+    """DOCK_TUNE_SHARD (multi-GPU block sharding), every rank emulated on this GPU: each rank clusters the whole
+    unit range (deterministically: every rank must get the same block order), docks the blocks rank, rank +
+    world, ... and writes only its units' rows of an INT32_MIN-filled buffer; the elementwise int32 MAX over the
+    ranks' buffers equals the single-GPU result bitwise, and every row was written by exactly one rank."""
+    P, m = 4, 4
+    R = g.receptor_ftmap_like((48, 40, 37), P)
+    w = g.weights(P)
+    probes = g.probes(7, m, P)
+    rot = g.rotations(90)   # 630 units = 5 blocks (a rank may own none at world = 8)
+    n = len(probes) * len(rot)
+    ctx = _ctx(D, R, w, m, 2)
+    ref = D.dock_probe_batch(ctx, probes, rot, k=4, rho=1)
+    import torch
+    bufs = []
+    for r in range(world):   # device output: rows of other ranks' units keep the INT32_MIN fill
+        D.dock_set_tuning(ctx, D.DOCK_TUNE_SHARD, (world << 16) | r)
+        out = torch.full((n, 4, 4), -2 ** 31, dtype=torch.int32, device="cuda")
+        D.dock_probe_batch(ctx, probes, rot, k=4, rho=1, out=out)
+        D.dock_sync(ctx)
+        bufs.append(out.cpu().numpy())
+    D.dock_set_tuning(ctx, D.DOCK_TUNE_SHARD, 1 << 16)
+    ctx.close()
+    written = np.stack([(b != np.iinfo(np.int32).min).any(axis=(1, 2)) for b in bufs])
+    assert (written.sum(0) == 1).all()
+    comb = np.maximum.reduce(bufs)
+    assert np.array_equal(comb, ref.view(np.int32).reshape(n, 4, 4))
+
+
 @pytest.mark.parametrize("engine", ENGINES)
 @pytest.mark.parametrize("rho,k", [(0, 4), (1, 4), (0, 1)])
 def test_integer_inputs_exact_poses(D, orc, rho, k, engine):

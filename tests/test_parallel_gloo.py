@@ -66,6 +66,45 @@ def test_sharded_equals_single_rank(orc, world, n_rot):
     assert all(np.array_equal(res[r], ref) for r in range(world))
 
 
+def _worker_rot(rank, world, port, n_rot, q):
+    os.environ.update(MASTER_ADDR="127.0.0.1", MASTER_PORT=str(port))
+    dist.init_process_group("gloo", rank=rank, world_size=world)
+    try:
+        from paper_conf_ipps_sukhwanih10_b200 import parallel
+        R = g.receptor_ftmap_like((16, 16, 16), 2)
+        w = g.weights(2)
+        probes = g.probes(3, 3, 2)
+        rot = g.rotations(n_rot)
+        full = parallel.dock_sharded_rotations(
+            lambda r0, r1: _oracle_block(R, w, probes, rot[r0:r1], 3, 1, 0, len(probes) * (r1 - r0)),
+            len(probes), n_rot, 3)
+        q.put((rank, full.numpy()))
+    finally:
+        dist.destroy_process_group()
+
+
+@pytest.mark.parametrize("world,n_rot", [(2, 5), (3, 7), (3, 2)])
+def test_rotation_sharded_equals_single_rank(orc, world, n_rot):
+    """The product path's rotation sharding (every rank docks every probe over its rotation slice, the
+    all-gather reorders into the global probe-major order and globalises the rotation indices) equals the
+    single-rank result; (3, 2): one rank owns no rotation and still joins the all-gather."""
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    port = _free_port()
+    procs = [ctx.Process(target=_worker_rot, args=(r, world, port, n_rot, q)) for r in range(world)]
+    for p in procs:
+        p.start()
+    res = dict(q.get(timeout=300) for _ in procs)
+    for p in procs:
+        p.join(timeout=60)
+        assert p.exitcode == 0
+    R = g.receptor_ftmap_like((16, 16, 16), 2)
+    probes = g.probes(3, 3, 2)
+    rot = g.rotations(n_rot)
+    ref = _oracle_block(R, g.weights(2), probes, rot, 3, 1, 0, len(probes) * n_rot).numpy()
+    assert all(np.array_equal(res[r], ref) for r in range(world))
+
+
 def test_shard_ranges_cover_exactly():
     from paper_conf_ipps_sukhwanih10_b200 import parallel
     for n in (1, 7, 8000, 70000):
