@@ -177,7 +177,7 @@ typedef enum {
                                      other one. */
     DOCK_TUNE_TC_EPILOGUE_WARPS = 6, /* tcgen05 epilogue warps: 0 auto (= the compiled maximum, 8), 4 or 8 (values
                                      above the compiled maximum are clamped to it) */
-    DOCK_TUNE_TC_CHUNK = 7,       /* tcgen05 variant 1: tiles per dynamically scheduled chunk (0 = auto, 4;
+    DOCK_TUNE_TC_CHUNK = 7,       /* tcgen05 variant 1: tiles per dynamically scheduled chunk (0 = auto, 4..16 by launch length;
                                      1..4096); one persistent CTA per SM takes chunks from a device counter */
     DOCK_TUNE_TC_SCHEDULE = 8,    /* tcgen05 variant 1 schedule.  A ring stage (4 K-steps of 16 products per accumulator)
                                      whose probe weights are zero for all 128 rotations of a block adds exact zeros, so a
