@@ -1410,6 +1410,7 @@ struct ClusterBinsSmem {
     int rec_cnt[CB_MAXREC];   //               units taken
     int rec_pos[CB_MAXREC];   //               block position of the first one
     uint16_t umask[CL_W];     // the window's unit masks
+    int wcnt[32][256];        // parallel stable sort (<= 256 distinct masks): per (warp, list entry) counts / offsets
 };
 __global__ void __launch_bounds__(1024, 1) k_tc_cluster_bins(const unsigned long long* __restrict__ masks, int n_slots,
                                                              int* __restrict__ sorted, int* __restrict__ perm)
@@ -1449,6 +1450,7 @@ __global__ void __launch_bounds__(1024, 1) k_tc_cluster_bins(const unsigned long
         for (int k = 0; k < PER; k++) {
             const int b = lane * PER + k, c = S.hist[b];
             S.fill[b] = run;
+            S.fill[b] = c ? li : -1;   // mask -> list entry (the parallel sort below); the serial one resets it
             if (c) {
                 S.lmask[li] = static_cast<uint16_t>(b);
                 S.lrem[li] = c;
@@ -1459,9 +1461,45 @@ __global__ void __launch_bounds__(1024, 1) k_tc_cluster_bins(const unsigned long
             run += c;
         }
         if (lane == 31) s_nl = inz;
-        // stable counting sort: units in index order, 32 at a time (lanes with equal masks ranked by lane), so
-        // the permutation is a deterministic function of the masks (block sharding needs every rank to compute
-        // the same one)
+    }
+    __syncthreads();
+    // stable counting sort (units of one mask in index order), so the permutation is a deterministic function of
+    // the masks -- block sharding needs every rank to compute the same one
+    if (s_nl <= 256) {
+        // parallel: warp w ranks its contiguous chunk; per-(warp, entry) counts, scanned over the warps
+        const int C = (n + 31) / 32, i_lo = warp * C, i_hi = min(n, i_lo + C), nl = s_nl;
+        for (int j = lane; j < nl; j += 32) S.wcnt[warp][j] = 0;
+        __syncwarp();
+        for (int i0 = i_lo; i0 < i_hi; i0 += 32) {
+            const int i = i0 + lane;
+            const int e = i < i_hi ? S.fill[S.umask[i]] : -1;
+            const unsigned grp = __match_any_sync(0xffffffffu, e);
+            if (i < i_hi && (grp & ((1u << lane) - 1u)) == 0u) S.wcnt[warp][e] += __popc(grp);
+            __syncwarp();
+        }
+        __syncthreads();
+        for (int j = tid; j < nl; j += blockDim.x) {   // exclusive scan over the warps, plus the entry's base
+            int run = S.lbase[j];
+            for (int w = 0; w < 32; w++) {
+                const int t = S.wcnt[w][j];
+                S.wcnt[w][j] = run;
+                run += t;
+            }
+        }
+        __syncthreads();
+        for (int i0 = i_lo; i0 < i_hi; i0 += 32) {
+            const int i = i0 + lane;
+            const int e = i < i_hi ? S.fill[S.umask[i]] : -1;
+            const unsigned grp = __match_any_sync(0xffffffffu, e);
+            const int rank = __popc(grp & ((1u << lane) - 1u));
+            if (i < i_hi) srt[S.wcnt[warp][e] + rank] = w0 + i;
+            __syncwarp();
+            if (i < i_hi && rank == 0) S.wcnt[warp][e] += __popc(grp);
+            __syncwarp();
+        }
+    } else if (warp == 0) {
+        // serial (one warp): units in index order, 32 at a time (lanes with equal masks ranked by lane)
+        for (int b = lane; b < CB_N; b += 32) S.fill[b] = S.hist[b];
         __syncwarp();
         for (int i0 = 0; i0 < n; i0 += 32) {
             const int i = i0 + lane;
@@ -1545,7 +1583,9 @@ __global__ void __launch_bounds__(1024, 1) k_tc_cluster_bins(const unsigned long
                 for (int e = 0; e < E; e++)
                     if (rem[e] > 0) {
                         const unsigned add = static_cast<unsigned>(__popc(msk[e] & ~U));
-                        const unsigned ratio = add * 1024u / static_cast<unsigned>(min(rem[e], room));
+                        // add * 1024 / take through the reciprocal (no integer division in the warp's hot loop)
+                        const unsigned ratio = static_cast<unsigned>(
+                            __fmul_rz(static_cast<float>(add * 1024u), __frcp_rn(static_cast<float>(min(rem[e], room)))));
                         best = min(best, (ratio << 16) | static_cast<unsigned>(lane * E + e));
                     }
                 best = __reduce_min_sync(0xffffffffu, best);
