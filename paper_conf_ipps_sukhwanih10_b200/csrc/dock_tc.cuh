@@ -1516,107 +1516,103 @@ __global__ void __launch_bounds__(1024, 1) k_tc_cluster_bins(const unsigned long
         }
     }
     __syncthreads();
-    if (warp == 0 && s_nl <= 32 * 8) {
-        // the greedy over <= 256 distinct masks with the list in registers: lane L owns entries [8L, 8L + 8)
-        constexpr int E = 8;
-        const int nl = s_nl;
-        unsigned msk[E];
-        int rem[E], base[E];
-#pragma unroll
-        for (int e = 0; e < E; e++) {
-            const int j = lane * E + e;
-            msk[e] = j < nl ? static_cast<unsigned>(S.lmask[j]) : 0u;
-            rem[e] = j < nl ? S.lrem[j] : 0;
-            base[e] = j < nl ? S.lbase[j] : 0;
-        }
-        unsigned U = 0;
-        int fill = 0, out = 0, nrec = 0, left = n;
-        while (left > 0) {
-            // zero-cost masks in list order, as many units as fit
-            const int cap = ROT - fill;
-            int cz = 0;
-#pragma unroll
-            for (int e = 0; e < E; e++) cz += (rem[e] > 0 && (msk[e] & ~U) == 0u) ? rem[e] : 0;
-            int incl = cz;
-            for (int d = 1; d < 32; d <<= 1) {
-                const int t = __shfl_up_sync(0xffffffffu, incl, d);
-                if (lane >= d) incl += t;
-            }
-            int before = incl - cz, ntake = 0;
-            int tk[E];
-#pragma unroll
-            for (int e = 0; e < E; e++) {
-                const int c = (rem[e] > 0 && (msk[e] & ~U) == 0u) ? rem[e] : 0;
-                tk[e] = max(0, min(c, cap - before));
-                before += c;
-                ntake += tk[e] > 0;
-            }
-            int rinc = ntake;
-            for (int d = 1; d < 32; d <<= 1) {
-                const int t = __shfl_up_sync(0xffffffffu, rinc, d);
-                if (lane >= d) rinc += t;
-            }
-            int r = nrec + rinc - ntake, pos = out + fill + (incl - cz);
-#pragma unroll
-            for (int e = 0; e < E; e++) {
-                if (tk[e] > 0) {
-                    S.rec_src[r] = base[e];
-                    S.rec_cnt[r] = tk[e];
-                    S.rec_pos[r] = pos;
-                    r++;
-                    rem[e] -= tk[e];
-                    base[e] += tk[e];
+    if (s_nl <= 256) {
+        // the greedy over <= 256 distinct masks, one list entry per thread of warps 0-7 (named barrier 1): per pass
+        // a block-wide prefix of the zero-cost units (as many as fit, in list order), then the mask that adds the
+        // fewest stages per unit it brings in (ties: the lowest entry = the lowest mask).  Every thread keeps
+        // the same block state (union, fill, ...) in registers; the per-warp partials are double-buffered by
+        // pass parity.  ~4 barriers of 8 warps per pass (one warp running the whole greedy took 120 us at
+        // prod: ~400 dependent instructions per pass).  In a host model of the prod workload the ratio rule
+        // cuts the blocks' active stages from 65.1 % to 63.4 % against "fewest stages" alone.
+        if (warp < 8) {
+            const int nl = s_nl, j = tid;
+            const unsigned mk = j < nl ? static_cast<unsigned>(S.lmask[j]) : 0u;
+            int rem = j < nl ? S.lrem[j] : 0, base = j < nl ? S.lbase[j] : 0;
+            __shared__ int s_wsum[2][8], s_wcnt[2][8];
+            __shared__ unsigned s_wmin[2][8];
+            __shared__ int s_wt;
+            __shared__ unsigned s_wm;
+            auto bar8 = []() { asm volatile("bar.sync 1, 256;" ::: "memory"); };
+            unsigned U = 0;
+            int fill = 0, out = 0, nrec = 0, left = n;
+            for (int ps = 0; left > 0; ps ^= 1) {
+                const int cap = ROT - fill;
+                // zero-cost units: block prefix in list order, capped at the room left
+                const int z = (rem > 0 && (mk & ~U) == 0u) ? rem : 0;
+                int incl = z;
+                for (int d = 1; d < 32; d <<= 1) {
+                    const int t = __shfl_up_sync(0xffffffffu, incl, d);
+                    if (lane >= d) incl += t;
                 }
-                pos += tk[e];
-            }
-            nrec += __shfl_sync(0xffffffffu, rinc, 31);
-            const int taken = min(__shfl_sync(0xffffffffu, incl, 31), cap);
-            fill += taken;
-            left -= taken;
-            if (fill < ROT && left > 0) {
-                // the mask that adds the fewest stages per unit it brings into the block (ties: the lowest entry
-                // = the lowest mask); in a host model of the prod workload this cuts the blocks' active stages
-                // from 65.1 % to 63.4 % against "fewest stages" alone
-                unsigned best = 0xffffffffu;
-                const int room = ROT - fill;
-#pragma unroll
-                for (int e = 0; e < E; e++)
-                    if (rem[e] > 0) {
-                        const unsigned add = static_cast<unsigned>(__popc(msk[e] & ~U));
-                        // add * 1024 / take through the reciprocal (no integer division in the warp's hot loop)
+                if (lane == 31) s_wsum[ps][warp] = incl;
+                bar8();
+                int before = incl - z, tz = 0;
+                for (int w = 0; w < 8; w++) {
+                    const int v = s_wsum[ps][w];
+                    if (w < warp) before += v;
+                    tz += v;
+                }
+                const int take = z > 0 ? max(0, min(z, cap - before)) : 0;
+                const unsigned tb = __ballot_sync(0xffffffffu, take > 0);
+                if (lane == 0) s_wcnt[ps][warp] = __popc(tb);
+                bar8();
+                int rbase = nrec, tr = 0;
+                for (int w = 0; w < 8; w++) {
+                    const int v = s_wcnt[ps][w];
+                    if (w < warp) rbase += v;
+                    tr += v;
+                }
+                if (take > 0) {
+                    const int r = rbase + __popc(tb & ((1u << lane) - 1u));
+                    S.rec_src[r] = base;
+                    S.rec_cnt[r] = take;
+                    S.rec_pos[r] = out + fill + before;
+                    rem -= take;
+                    base += take;
+                }
+                const int taken = min(tz, cap);
+                fill += taken;
+                left -= taken;
+                nrec += tr;
+                if (fill < ROT && left > 0) {
+                    const int room = ROT - fill;
+                    unsigned key = 0xffffffffu;
+                    if (rem > 0) {
+                        const unsigned add = static_cast<unsigned>(__popc(mk & ~U));
                         const unsigned ratio = static_cast<unsigned>(
-                            __fmul_rz(static_cast<float>(add * 1024u), __frcp_rn(static_cast<float>(min(rem[e], room)))));
-                        best = min(best, (ratio << 16) | static_cast<unsigned>(lane * E + e));
+                            __fmul_rz(static_cast<float>(add * 1024u), __frcp_rn(static_cast<float>(min(rem, room)))));
+                        key = (ratio << 16) | static_cast<unsigned>(j);
                     }
-                best = __reduce_min_sync(0xffffffffu, best);
-                const int j = static_cast<int>(best & 0xffffu), owner = j / E, ej = j % E;
-                int take = 0;
-                unsigned mj = 0;
-#pragma unroll
-                for (int e = 0; e < E; e++)
-                    if (lane == owner && e == ej) {
-                        take = min(rem[e], ROT - fill);
-                        S.rec_src[nrec] = base[e];
-                        S.rec_cnt[nrec] = take;
+                    key = __reduce_min_sync(0xffffffffu, key);
+                    if (lane == 0) s_wmin[ps][warp] = key;
+                    bar8();
+                    unsigned win = 0xffffffffu;
+                    for (int w = 0; w < 8; w++) win = min(win, s_wmin[ps][w]);
+                    if (j == static_cast<int>(win & 0xffffu)) {
+                        const int t = min(rem, room);
+                        S.rec_src[nrec] = base;
+                        S.rec_cnt[nrec] = t;
                         S.rec_pos[nrec] = out + fill;
-                        rem[e] -= take;
-                        base[e] += take;
-                        mj = msk[e];
+                        rem -= t;
+                        base += t;
+                        s_wt = t;
+                        s_wm = mk;
                     }
-                take = __shfl_sync(0xffffffffu, take, owner);
-                mj = __shfl_sync(0xffffffffu, mj, owner);
-                nrec++;
-                U |= mj;
-                fill += take;
-                left -= take;
+                    bar8();
+                    U |= s_wm;
+                    fill += s_wt;
+                    left -= s_wt;
+                    nrec++;
+                    bar8();   // s_wt / s_wm are rewritten in the next pass
+                }
+                if (fill == ROT || left == 0) {
+                    out += ROT;
+                    fill = 0;
+                    U = 0;
+                }
             }
-            if (fill == ROT || left == 0) {
-                out += ROT;
-                fill = 0;
-                U = 0;
-            }
+            if (tid == 0) s_nrec = nrec;
         }
-        if (lane == 0) s_nrec = nrec;
     } else if (warp == 0) {
         // the greedy over the distinct masks (one warp; list entries lane, lane + 32, ...)
         const int nl = s_nl;
