@@ -356,6 +356,32 @@ def test_tc_occupancy_schedule_modes(D, orc):
     assert mism == 0
 
 
+def test_tc_occupancy_schedule_two_windows(D, orc):
+    """More units than one clustering window (8192): two windows are clustered independently, blocks never
+    straddle them, and the clustered schedule's poses equal the dense schedule's bitwise; sampled units of
+    both windows validate against the oracle."""
+    P, m = 4, 4
+    R = g.receptor_ftmap_like((48, 40, 37), P)
+    w = g.weights(P)
+    probes = g.probes(17, m, P)
+    rot = g.rotations(500)   # 8500 units
+    n = len(probes) * len(rot)
+    ctx = _ctx(D, R, w, m, 2)
+    D.dock_set_tuning(ctx, D.DOCK_TUNE_TC_SCHEDULE, 2)
+    dense = D.dock_probe_batch(ctx, probes, rot, k=4, rho=1)
+    D.dock_set_tuning(ctx, D.DOCK_TUNE_TC_SCHEDULE, 0)
+    clus = D.dock_probe_batch(ctx, probes, rot, k=4, rho=1)
+    info = D.dock_get_info(ctx)
+    ctx.close()
+    assert info["tc_variant_last"] == 1 and info["tc_ksteps_exec_last"] < 48.0
+    for f in ("rot", "t_lin"):
+        assert np.array_equal(clus[f], dense[f])
+    assert np.array_equal(clus["score"].view(np.uint32), dense["score"].view(np.uint32))
+    units = [0, 4000, 8191, 8192, 8300, n - 1]
+    for u, (S, A) in zip(units, _oracle_units(orc, R, w, probes, rot, units)):
+        validate_unit(S, A, clus[u]["t_lin"], clus[u]["score"], 4, 1)   # raises on a violation (ties may differ)
+
+
 def test_tc_occupancy_schedule_integer_exact(D, orc):
     """Clustered occupancy schedule (> 128 units; m = 3 and 2 on the mask histogram, m = 5 on the unit greedy
     where variant 1 runs it) on integer inputs: poses equal the FP64 oracle exactly, ties included (P9)."""
