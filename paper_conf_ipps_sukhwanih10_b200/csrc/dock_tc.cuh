@@ -242,10 +242,12 @@ __device__ __forceinline__ void list_insert(unsigned long long (&L)[LIST], unsig
 
 // One 32-value chunk of scores (rotation of this thread, translations tbase + c0 + j, j < jmax valid)
 // into the per-thread exact top-LIST list; GRID writes the chunk to the score grid instead.
+// tgk: the unit's global pruning bound T read during the kernel (keys above it can never be among the picks,
+// DESIGN.md §8), so (th, th_t) is the smaller of the list's last key and tgk.
 template <bool GRID>
 __device__ __forceinline__ void epi_chunk(const uint32_t (&v)[32], unsigned long long (&lst)[LIST], float& th,
                                           uint32_t& th_t, uint32_t tbase, int c0, int jmax, float* grid_row,
-                                          unsigned* nins = nullptr)
+                                          unsigned* nins = nullptr, unsigned long long tgk = KEY_MAX)
 {
     if constexpr (GRID) {
 #pragma unroll
@@ -268,17 +270,19 @@ __device__ __forceinline__ void epi_chunk(const uint32_t (&v)[32], unsigned long
             uint32_t msk = 0;
 #pragma unroll
             for (int j = 0; j < 32; j++) msk |= (__uint_as_float(v[j]) <= th && j < jmax) ? (1u << j) : 0u;
+            unsigned long long lim = lst[LIST - 1] < tgk ? lst[LIST - 1] : tgk;
             while (msk) {
                 const int j = __ffs(msk) - 1;
                 msk &= msk - 1;
                 const float sv = __uint_as_float(select32(v, j));
                 if (sv <= th) {
                     const unsigned long long key = dk::make_key(sv, tbase + c0 + j);
-                    if (key < lst[LIST - 1]) {
+                    if (key < lim) {
                         if (nins) ++nins[0];
                         list_insert(lst, key);
-                        th = dk::key_score_bound(static_cast<uint32_t>(lst[LIST - 1] >> 32));
-                        th_t = static_cast<uint32_t>(lst[LIST - 1] & 0xffffffffu);
+                        lim = lst[LIST - 1] < tgk ? lst[LIST - 1] : tgk;
+                        th = dk::key_score_bound(static_cast<uint32_t>(lim >> 32));
+                        th_t = static_cast<uint32_t>(lim & 0xffffffffu);
                     }
                 }
             }
@@ -289,6 +293,30 @@ __device__ __forceinline__ void epi_chunk(const uint32_t (&v)[32], unsigned long
 // Item end: bound T_w from k list entries pairwise farther than 2*rho apart, then
 // publish bound, mu and the keys <= T (k_merge finishes the greedy).  Loops over the register list
 // are fully unrolled (static indices keep it in registers).
+// T_w of a list: the key of the k-th entry of a greedy pick from the list with pairwise cyclic Chebyshev distance
+// > 2 rho (any k such points bound the true greedy's k-th pick); KEY_MAX if there are fewer.
+__device__ __forceinline__ unsigned long long list_bound(const unsigned long long (&lst)[LIST], const TcArgs& a)
+{
+    unsigned long long Tw = KEY_MAX;
+    uint32_t chosen[32];
+    int nc = 0;
+#pragma unroll
+    for (int i = 0; i < LIST; i++) {
+        const unsigned long long key = lst[i];
+        if (key != KEY_MAX && nc < a.k) {
+            const uint32_t t = static_cast<uint32_t>(key & 0xffffffffu);
+            bool far = true;
+            for (int c = 0; c < nc; c++) far = far && dk::cheb_cyc(t, chosen[c], a.nx, a.ny, a.nz) > 2 * a.rho;
+            if (far) {
+                chosen[nc] = t;
+                nc++;
+                if (nc == a.k) Tw = key;
+            }
+        }
+    }
+    return Tw;
+}
+
 __device__ __forceinline__ void epi_publish(const unsigned long long (&lst)[LIST], int slot, const TcArgs& a)
 {
     unsigned long long Tw = KEY_MAX;
@@ -333,7 +361,7 @@ __device__ __forceinline__ void epi_tile(const TcArgs& a, uint32_t tmem, uint64_
                                          int nclass, int lane, int slot, bool rot_ok, int tx, int ty, int tz,
                                          unsigned long long (&lst)[LIST], float& th, uint32_t& th_t, bool tr,
                                          long long& tw0, long long& tw1, uint64_t* row_full = nullptr,
-                                         unsigned row_ph = 0, unsigned* nins = nullptr)
+                                         unsigned row_ph = 0, unsigned* nins = nullptr, unsigned long long tgk = KEY_MAX)
 {
     constexpr int NCH = NTT / 32;
     const int x0 = tx * NTT;
@@ -366,8 +394,8 @@ __device__ __forceinline__ void epi_tile(const TcArgs& a, uint32_t tmem, uint64_
             if (lane == 0) dk::mbar_arrive(&tm_empty[q]);
             if (!row_ok) continue;
             float* grow = GRID ? a.grid + static_cast<size_t>(slot) * a.nx * a.ny * a.nz + tbase : nullptr;
-            epi_chunk<GRID>(v0, lst, th, th_t, tbase, c0, min(32, a.nx - x0 - c0), grow, nins);
-            epi_chunk<GRID>(v1, lst, th, th_t, tbase, c1, min(32, a.nx - x0 - c1), grow, nins);
+            epi_chunk<GRID>(v0, lst, th, th_t, tbase, c0, min(32, a.nx - x0 - c0), grow, nins, tgk);
+            epi_chunk<GRID>(v1, lst, th, th_t, tbase, c1, min(32, a.nx - x0 - c1), grow, nins, tgk);
             continue;
         }
 #pragma unroll 1
@@ -384,7 +412,8 @@ __device__ __forceinline__ void epi_tile(const TcArgs& a, uint32_t tmem, uint64_
             }
             if (!row_ok) continue;
             epi_chunk<GRID>(v, lst, th, th_t, tbase, c0, min(32, a.nx - x0 - c0),
-                            GRID ? a.grid + static_cast<size_t>(slot) * a.nx * a.ny * a.nz + tbase : nullptr);
+                            GRID ? a.grid + static_cast<size_t>(slot) * a.nx * a.ny * a.nz + tbase : nullptr, nullptr,
+                            tgk);
         }
     }
 }
@@ -909,8 +938,10 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
             unsigned long long lst[LIST];
 #pragma unroll
             for (int i = 0; i < LIST; i++) lst[i] = KEY_MAX;
-            float th = __int_as_float(0x7f800000);   // score of the list's last key (+inf while not full)
-            uint32_t th_t = 0xffffffffu;             // t_lin of the list's last key
+            float th = __int_as_float(0x7f800000);   // score of the gate key: min(list's last key, tgk) (+inf: none)
+            uint32_t th_t = 0xffffffffu;             // t_lin of the gate key
+            unsigned long long tgk = KEY_MAX;        // the unit's pruning bound T as last read
+            int since = 0;                            // tiles of the current block (periodic bound publish)
             int ti = 0;                               // tiles so far (TMEM phases)
             long long g, tpub = 0;
             unsigned nins[3] = {0, 0, 0};
@@ -930,6 +961,8 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                     for (int i = 0; i < LIST; i++) lst[i] = KEY_MAX;
                     th = __int_as_float(0x7f800000);
                     th_t = 0xffffffffu;
+                    tgk = KEY_MAX;
+                    since = 0;
                     cur = blk;
                     const int pos = static_cast<int>(gblock(blk)) * ROT + r;   // position in the block order
                     rot_ok = pos < n_eff;
@@ -938,8 +971,23 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_tc(const __grid_constant__
                 const int t0 = static_cast<int>(g % a.ntiles);
                 int tx = t0 % a.ntx, ty = (t0 / a.ntx) % a.nty, tz = t0 / (a.ntx * a.nty);
                 for (int j = 0; j < n; j++, ti++) {
+                    if (!GRID && rot_ok) {
+                        // the unit's pruning bound T so far (other lists' published T_w): keys above it cannot be
+                        // picks, so the gate also skips them (fewer insertions; DESIGN.md §8 stays exact)
+                        const unsigned long long tg = *reinterpret_cast<volatile unsigned long long*>(&a.T[slot]);
+                        if (tg < tgk) {
+                            tgk = tg;
+                            const unsigned long long lim = lst[LIST - 1] < tgk ? lst[LIST - 1] : tgk;
+                            th = dk::key_score_bound(static_cast<uint32_t>(lim >> 32));
+                            th_t = static_cast<uint32_t>(lim & 0xffffffffu);
+                        }
+                        if ((++since & 31) == 0) {   // publish this list's bound every 32 tiles
+                            const unsigned long long tw = list_bound(lst, a);
+                            if (tw < tgk) atomicMin(&a.T[slot], tw);
+                        }
+                    }
                     epi_tile<NT, Q, GRID>(a, tmem, tm_empty, quarter, cls, nclass, lane, slot, rot_ok, tx, ty, tz, lst,
-                                          th, th_t, tr, tw0, tw1, tm_full, ti & 1, tr ? nins : nullptr);
+                                          th, th_t, tr, tw0, tw1, tm_full, ti & 1, tr ? nins : nullptr, tgk);
                     if (++tx == a.ntx) {
                         tx = 0;
                         if (++ty == a.nty) {
