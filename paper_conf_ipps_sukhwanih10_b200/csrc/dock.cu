@@ -107,6 +107,8 @@ struct dock_ctx {
     int shard_rank = 0, shard_world = 1;   // DOCK_TUNE_SHARD: block sharding of the variant-1 block order
     int tc_nblk_local = -1;    // blocks of the last main pass this rank docks (-1: all)
     DevBuf tc_blkmap, tc_owned;
+    int sp_bound_every = 2;    // sparse engine: columns between global-bound refreshes (0 / 1 / 2 / 4 / 8 -> c64 0.517 / 0.457 /
+                               // 0.441 / 0.477 / 0.517 ms, large shard 36.0 / 35.3 / 33.2 / 32.8 / 35.6 ms); DOCK_SP_BOUND_EVERY overrides
     int tc_seg_cost = 8;       // per-tile cost of a chunk beyond its ring stages, in ring stages (prod: 0 / 3 / 6 /
                                // 9 / 12 / 24 -> 12.20 / 11.79 / 11.40 / 11.35 / 11.48 / 11.84 ms); DOCK_TC_SEG_COST
                                // (environment) overrides it
@@ -985,6 +987,7 @@ sp::SpArgs sp_args(dock_ctx* ctx, const SpCall& sc, const sp::Group* d_groups, i
 {
     const SpPlan& pl = ctx->spplan[sc.m][sc.xts];
     sp::SpArgs a{};
+    a.bound_every = ctx->sp_bound_every;
     a.nx = ctx->nx;
     a.ny = ctx->ny;
     a.nz = ctx->nz;
@@ -1583,6 +1586,7 @@ dock_status dock_init(const dock_grid_desc* g, const float* receptor, const floa
         if (cudaEventCreateWithFlags(&st.ev, cudaEventDisableTiming) != cudaSuccess) return bail(DOCK_E_CUDA);
     if (const char* e = getenv("DOCK_FB_HOST_LOOP")) ctx->fb_host_loop = atoi(e);
     if (const char* e = getenv("DOCK_TC_SEG_COST")) ctx->tc_seg_cost = std::max(0, atoi(e));   // tuning experiments
+    if (const char* e = getenv("DOCK_SP_BOUND_EVERY")) ctx->sp_bound_every = std::max(0, atoi(e));
     if (const char* e = getenv("DOCK_TC_TRACE")) {
         if (atoi(e) > 0 && cudaMalloc(&ctx->d_trace, sizeof(unsigned long long) * tc::TR_N) != cudaSuccess)
             return bail(DOCK_E_OOM);

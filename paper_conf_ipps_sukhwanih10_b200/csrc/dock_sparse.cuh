@@ -63,6 +63,7 @@ struct SpArgs {
     int slot_words;             // plane slot stride (floats, 128-B aligned)
     int npl;                    // plane-ring depth (slots per atom)
     int cols_per_item;          // columns (TX x TY x all nz translations) per item; lists persist across them
+    int bound_every;            // columns between refreshes of the lists' global pruning bound (0: never)
     int G;                      // items per group = ceil(ntx * nty / cols_per_item)
     int box_bytes;              // TXB * TYB * 4
     const Group* groups;        // [n_groups]
@@ -246,12 +247,15 @@ struct Vec {   // passed by value to the out-of-line helpers (a pointer would fo
     float v[N];
 };
 
+// tg: the unit's pruning bound T as last read (keys above it can never be picks): the gate key is
+// min(list's 32nd key, tg).
 template <int XTS, int ZT>
 __device__ __noinline__ void sp_insert(unsigned long long* L, float2* th_rec, const Vec<XTS * ZT> acc, unsigned vmask,
-                                       uint32_t tbase, uint32_t plane_stride, int lane)
+                                       uint32_t tbase, uint32_t plane_stride, int lane, unsigned long long tg)
 {
     unsigned long long lst = L[lane];
     unsigned long long thk = dk::shfl_u64(lst, 31);
+    thk = thk < tg ? thk : tg;
 #pragma unroll
     for (int v = 0; v < XTS * ZT; v++) {
         const uint32_t t = tbase + static_cast<uint32_t>(v / XTS) * plane_stride + 32u * static_cast<uint32_t>(v % XTS);
@@ -261,15 +265,38 @@ __device__ __noinline__ void sp_insert(unsigned long long* L, float2* th_rec, co
             const int src = __ffs(mm) - 1;
             dk::warp_list_insert(lst, dk::shfl_u64(key, src), lane);
             thk = dk::shfl_u64(lst, 31);
+            thk = thk < tg ? thk : tg;
             mm &= ~(1u << src);
             mm &= __ballot_sync(FULL, key < thk);
         }
     }
     L[lane] = lst;
-    if (lane == 31)   // gate record of the list: score bound and t_lin of its 32nd key
-        *th_rec = make_float2(dk::key_score_bound(static_cast<uint32_t>(lst >> 32)),
-                              __uint_as_float(static_cast<uint32_t>(lst & 0xffffffffu)));
+    if (lane == 31) {   // gate record of the list: score bound and t_lin of min(its 32nd key, tg)
+        const unsigned long long g = lst < tg ? lst : tg;
+        *th_rec = make_float2(dk::key_score_bound(static_cast<uint32_t>(g >> 32)),
+                              __uint_as_float(static_cast<uint32_t>(g & 0xffffffffu)));
+    }
     __syncwarp();
+}
+
+// T_w of a warp list (lane i holds its i-th smallest key): the key of the k-th entry of a greedy pick with
+// pairwise cyclic Chebyshev distance > 2 rho; KEY_MAX if there are fewer.  Warp-uniform result.
+__device__ __forceinline__ unsigned long long sp_list_bound(unsigned long long key, int k, int rho, int nx, int ny,
+                                                            int nz)
+{
+    const uint32_t t = static_cast<uint32_t>(key & 0xffffffffu);
+    bool excl = (key == KEY_MAX);
+    unsigned long long Tw = KEY_MAX;
+    for (int j = 0; j < k; j++) {
+        const unsigned b = __ballot_sync(FULL, !excl);
+        if (!b) break;
+        const int f = __ffs(b) - 1;
+        const unsigned long long kf = dk::shfl_u64(key, f);
+        const uint32_t tf = static_cast<uint32_t>(kf & 0xffffffffu);
+        excl = excl || (dk::cheb_cyc(t, tf, nx, ny, nz) <= 2 * rho);
+        if (j == k - 1) Tw = kf;
+    }
+    return Tw;
 }
 
 // mbarrier wait on a 32-bit shared address (no generic-to-shared conversion in the loop)
@@ -333,7 +360,8 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
     __shared__ int s_dterm[TMAX * RB];   // [term][rotation]: direct term (vx | vy << 8 | vz << 16 | term << 24) or -1
     __shared__ int s_tmax, s_ndirect;    // most occupied voxels of a rotation of the group; direct terms in the group
     __shared__ unsigned long long s_lst[NWC][RBW][32];   // per warp and rotation: sorted top-32 keys (one per lane)
-    __shared__ float2 s_th[NWC][RBW];                     // per list: score bound and t_lin of its 32nd key
+    __shared__ float2 s_th[NWC][RBW];                     // per list: score bound and t_lin of the gate key
+    __shared__ unsigned long long s_tg[NWC][RBW];         // per list: the unit's pruning bound T as last read
 
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     const int grp = blockIdx.x / a.G, reg = blockIdx.x % a.G;
@@ -418,7 +446,10 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
     unsigned long long(*lists)[32] = s_lst[warp];
 #pragma unroll
     for (int r = 0; r < RBW; r++) lists[r][lane] = KEY_MAX;
-    if (lane < RBW) s_th[warp][lane] = make_float2(__int_as_float(0x7f800000), __uint_as_float(0xffffffffu));
+    if (lane < RBW) {
+        s_th[warp][lane] = make_float2(__int_as_float(0x7f800000), __uint_as_float(0xffffffffu));
+        s_tg[warp][lane] = KEY_MAX;
+    }
     __syncwarp();
     const uint32_t lane_base = dk::smem_u32(ring) + 4u * static_cast<uint32_t>(ry * a.TXB + lane);
     const uint32_t ring_bytes = static_cast<uint32_t>(npl * slot_bytes);
@@ -428,6 +459,32 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
     unsigned wphase = 0;
     int pslot = (pg * ZT) % npl;   // ring slot of this warp's first plane, maintained incrementally
     for (int c = c0; c < c1; c++, cbase += n_planes) {
+        if constexpr (!GRID) {
+            if (a.bound_every > 0 && c > c0 && (c - c0) % a.bound_every == 0) {
+                // publish each list's bound T_w and read back the unit's T: keys above T can never be picks
+                // (DESIGN.md §8), so the gate also skips them (fewer insertions, same poses)
+#pragma unroll 1
+                for (int r = 0; r < RBW && rbase + r < nrot; r++) {
+                    const int slot = gr.slot0 + rbase + r;
+                    const unsigned long long key = lists[r][lane];
+                    const unsigned long long tw = sp_list_bound(key, a.k, a.rho, a.nx, a.ny, a.nz);
+                    unsigned long long tg = 0;
+                    if (lane == 0) {
+                        const unsigned long long old = tw != KEY_MAX ? atomicMin(&a.T[slot], tw)
+                                                                     : *reinterpret_cast<volatile unsigned long long*>(&a.T[slot]);
+                        tg = old < tw ? old : tw;
+                        s_tg[warp][r] = tg;
+                    }
+                    const unsigned long long k31 = dk::shfl_u64(key, 31);
+                    if (lane == 0) {
+                        const unsigned long long gk = k31 < tg ? k31 : tg;
+                        s_th[warp][r] = make_float2(dk::key_score_bound(static_cast<uint32_t>(gk >> 32)),
+                                                    __uint_as_float(static_cast<uint32_t>(gk & 0xffffffffu)));
+                    }
+                }
+                __syncwarp();
+            }
+        }
         const int tx = c % a.ntx, ty = c / a.ntx;
         const int y = ty * TY + ry;
         const int xb = tx * a.TX + lane;
@@ -562,7 +619,8 @@ __global__ void __launch_bounds__(NTHREADS, 1) k_corr_sparse(const __grid_consta
                                 Vec<V> av;
 #pragma unroll
                                 for (int v = 0; v < V; v++) av.v[v] = acc[r][v];
-                                sp_insert<XTS, ZT>(lists[r], &s_th[warp][r], av, vmask, tbase, plane_stride, lane);
+                                sp_insert<XTS, ZT>(lists[r], &s_th[warp][r], av, vmask, tbase, plane_stride, lane,
+                                                   s_tg[warp][r]);
                             }
                         }
                     }
